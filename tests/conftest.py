@@ -1,0 +1,20 @@
+import os
+import sys
+
+import pytest
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+if ROOT not in sys.path:
+    sys.path.insert(0, ROOT)
+
+
+def pytest_configure(config):
+    config.addinivalue_line("markers", "gpu: needs a CUDA device (B200); run with -m gpu")
+    config.addinivalue_line("markers", "slow: long-running")
+
+
+def pytest_collection_modifyitems(config, items):
+    # tests under tests/gpu/ are GPU tests even if a marker was forgotten
+    for it in items:
+        if os.sep + "gpu" + os.sep in str(it.fspath) and "gpu" not in it.keywords:
+            it.add_marker(pytest.mark.gpu)
