@@ -1,0 +1,234 @@
+/*
+ * qudax.h — C ABI of the B200-native even-odd Wilson-clover Dslash / halo / mixed-precision
+ * BiCGstab library (the hot path of arXiv:1011.0024, "Parallelizing the QUDA Library for
+ * Multi-GPU Calculations in Lattice QCD"; PAPER.md line numbers cited as P:a-b).
+ *
+ * The paper's library exposes "a simple C interface to allow for easy integration with LQCD
+ * application software": the only large transfers are "the initial upload of the
+ * source vector to the GPU and the final download of the solution, aside from occasional
+ * small messages needed to complete global sums".  This header is that
+ * boundary.  Plain pointers and sizes only; no C++ or torch types.
+ *
+ * ---------------------------------------------------------------------------------------
+ * Conventions (all readings of the paper are listed in DESIGN.md "Readings")
+ * ---------------------------------------------------------------------------------------
+ * Lattice  global X x Y x Z x T (x fastest, t slowest); partitioned in T only into nranks
+ *          equal slabs: rank r owns global t in [r*T_loc,(r+1)*T_loc),
+ *          T_loc = T / nranks.  Requires X even, T_loc even (so local and global parity
+ *          agree), T_loc >= 2.  Site parity = (x + y + z + t_global) mod 2.
+ * Host gauge  const double[4][T_loc][Z][Y][X][3][3][2]: the rank's slab, U_mu(x) stored at x
+ *          (P:425-432), row-major 3x3 complex, mu = 0..3 <-> x, y, z, t.  Borrowed for the
+ *          duration of the call only.
+ * Host spinor double[T_loc][Z][Y][X][4][3][2] in the DeGrand-Rossi chiral basis (the
+ *          "conventional chiral basis" of eq. (6)).  Borrowed per call.
+ * Operator M_kappa = 2 kappa M(eq. (2)) = T - kappa D with T = 1 + 2 kappa A (clover A of
+ *          eq. (2); kappa = 1/(2(4+m))).  Even-odd: the solver works
+ *          on the asymmetric Schur complement on even sites
+ *              Mhat = T_ee - kappa^2 D_eo T_oo^{-1} D_oe,   Mhat^dag = gamma5 Mhat gamma5.
+ * Device spinor fields ("parity fields") are plain device buffers owned by the CALLER, of
+ *          qudax_spinor_bytes(ctx, prec) bytes, holding the V_h = V_loc/2 sites of one parity
+ *          in the library's site-major SoA layout (eq. (4): N_int/N_vec blocks of
+ *          V_h 16-byte short vectors; non-relativistic spin basis, eq. (6)).  Half precision
+ *          appends one float norm per site.  The layout is opaque to callers:
+ *          move data in and out with qudax_spinor_load/store.  Reductions never see ghost
+ *          zones: ghosts live in separate library-owned buffers.
+ *
+ * Precision / reconstruct: prec = bytes per stored real
+ *          (2 = 16-bit fixed point "half", 4 = fp32, 8 = fp64); recon = reals stored per link
+ *          (18 full, 12 two-row with row3 = conj(row1 x row2), 8 = two phases + u01,u02,u10).
+ *
+ * Ownership: the ctx owns every internal device allocation (through the dev_alloc/dev_free
+ *          hooks when given — the Python binding passes PyTorch's caching allocator — else
+ *          cudaMalloc) and its comm stream.  Host pointers are borrowed per call.
+ * Ordering: qudax_dslash / qudax_matpc / qudax_mdagm / qudax_spinor_load_dev are
+ *          stream-ordered on the ctx compute stream and return before the GPU finishes.
+ *          qudax_gauge_load, qudax_spinor_load/store (host), reductions and the solvers are
+ *          synchronous.
+ * Errors:  every call returns a qudax_status; no C++ exception crosses the ABI.  CUDA and NCCL
+ *          failures are sticky (the ctx must be finalized); qudax_last_error() explains.
+ * Threads: a ctx is not thread-safe.  With nranks > 1 every rank must make the same sequence
+ *          of calls (collective ordering rule).
+ */
+#ifndef QUDAX_H
+#define QUDAX_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define QUDAX_ABI_VERSION 1
+
+typedef enum {
+    QUDAX_OK = 0,
+    QUDAX_ERR_ARG = 1,           /* bad dims, parity, precision, null pointer, state mismatch */
+    QUDAX_ERR_STATE = 2,         /* call out of order (e.g. dslash before gauge_load) or sticky error */
+    QUDAX_ERR_CUDA = 3,          /* CUDA runtime failure (sticky) */
+    QUDAX_ERR_NCCL = 4,          /* NCCL failure (sticky) */
+    QUDAX_ERR_UNSUPPORTED = 5,   /* e.g. 8-reconstruct on near-singular links (reading Q6) */
+    QUDAX_ERR_NOT_CONVERGED = 6, /* solver hit maxiter; x holds the last iterate */
+    QUDAX_ERR_OOM = 7,           /* device allocation failed */
+    QUDAX_ERR_COMM = 8           /* host transport hook returned non-zero */
+} qudax_status;
+
+typedef enum { QUDAX_HALF = 2, QUDAX_SINGLE = 4, QUDAX_DOUBLE = 8 } qudax_prec;
+typedef enum { QUDAX_RECON_18 = 18, QUDAX_RECON_12 = 12, QUDAX_RECON_8 = 8 } qudax_recon;
+typedef enum { QUDAX_EVEN = 0, QUDAX_ODD = 1 } qudax_parity;
+
+/* What a single Dslash kernel computes on the output parity p (input field of parity 1-p):
+ *   HOP         out = D_{p,1-p} in                                   (1320 flops/site)
+ *   CLOVER_INV  out = T_pp^{-1} D_{p,1-p} in                         (+504, clover fused,
+ *                                                                      P:390-395)
+ *   CLOVER_XPAY out = T_pp x + a * D_{p,1-p} in                     (+504 +48)
+ * Mhat = [kernel CLOVER_INV on odd] then [kernel CLOVER_XPAY on even, a = -kappa^2]. */
+typedef enum { QUDAX_HOP = 0, QUDAX_CLOVER_INV = 1, QUDAX_CLOVER_XPAY = 2 } qudax_dslash_kind;
+
+/* Halo transport:
+ *   NONE  nranks must be 1; the Dslash wraps T periodically inside one kernel.
+ *   NCCL  ncclSend/ncclRecv of spin-projected faces on a comm stream, overlapped with the
+ *         interior kernel; ncclAllReduce for global sums.  With
+ *         nranks == 1 this is the loopback test mode (faces go through NCCL to self).
+ *   HOST  faces staged through pinned host memory and exchanged by the caller's hooks
+ *         (the paper's non-overlapped strategy); used to run several ranks on
+ *         one GPU in tests. */
+typedef enum { QUDAX_COMM_NONE = 0, QUDAX_COMM_NCCL = 1, QUDAX_COMM_HOST = 2 } qudax_comm_kind;
+
+typedef struct qudax_ctx qudax_ctx;
+
+/* Host transport hooks for QUDAX_COMM_HOST.  exchange: send send_fwd (bytes) to rank+1 and
+ * send_back to rank-1, receive from rank-1 into recv_back and from rank+1 into recv_fwd
+ * (periodic ring).  allreduce: in-place sum of n doubles over ranks.  Return 0 on success. */
+typedef int (*qudax_exchange_fn)(const void *send_fwd, const void *send_back, void *recv_back,
+                                 void *recv_fwd, size_t bytes, void *user);
+typedef int (*qudax_allreduce_fn)(double *vals, int n, void *user);
+typedef void *(*qudax_alloc_fn)(size_t bytes, void *user);
+typedef void (*qudax_free_fn)(void *ptr, void *user);
+
+typedef struct {
+    int global_dims[4];          /* X, Y, Z, T */
+    int nranks, rank, device;    /* device = CUDA ordinal this rank drives */
+    int comm;                    /* qudax_comm_kind */
+    int overlap;                 /* NCCL: 1 = interior kernel overlaps the halo,
+                                    0 = exchange first then one kernel */
+    const void *nccl_id;         /* QUDAX_COMM_NCCL: 128-byte ncclUniqueId from qudax_nccl_unique_id
+                                    on rank 0, broadcast by the caller */
+    uintptr_t stream;            /* compute cudaStream_t (e.g. torch current stream), 0 = own */
+    qudax_alloc_fn dev_alloc;    /* optional device allocator hooks (NULL = cudaMalloc) */
+    qudax_free_fn dev_free;
+    void *alloc_user;
+    qudax_exchange_fn host_exchange; /* QUDAX_COMM_HOST hooks */
+    qudax_allreduce_fn host_allreduce;
+    void *comm_user;
+} qudax_init_param;
+
+typedef struct {
+    int prec, recon;             /* outer ("high") precision copy of gauge + clover */
+    int prec_sloppy, recon_sloppy; /* inner ("sloppy") copy for reliable updates */
+    int t_boundary;              /* +1 periodic, -1 antiperiodic in T (reading Q5) */
+    double kappa, csw;           /* M_kappa = T - kappa D, T = 1 + 2 kappa A(csw) (readings Q1, Q4) */
+} qudax_gauge_param;
+
+typedef struct {
+    double tol;                  /* stop when the TRUE residual ||b - M x|| / ||b|| <= tol (Q9) */
+    double delta;                /* reliable-update threshold (Algorithm R) */
+    int maxiter;                 /* iteration cap; tol = 0 with maxiter = k runs exactly k iterations */
+    int prec_sloppy;             /* precision of the Krylov iteration (must have a gauge copy) */
+    int prec;                    /* outer precision of x, r and the reliable-update residual */
+    int use_schur;               /* 1: solve the full system M x = b via prepare/Mhat/reconstruct */
+} qudax_solve_param;
+
+typedef struct {
+    int iters, reliable_updates;
+    double true_res;             /* fp64 ||b - M x|| / ||b|| of the returned x (full system if use_schur) */
+    double true_res_schur;       /* fp64 ||bhat - Mhat x_e|| / ||bhat|| */
+    double secs;                 /* wall time of the call (includes H2D / D2H for the host entry) */
+    double flops;                /* effective flops (P:755-758 convention, reading Q16) */
+    double gflops;
+} qudax_solve_stats;
+
+/* Per-site work and traffic model, for reporting and tests. */
+typedef struct {
+    double flops;                /* effective flops per output site (reconstruction not counted) */
+    double bytes_paper;          /* paper model: every neighbour gather is memory traffic */
+    double bytes_compulsory;     /* each link / clover / spinor read once, output written once */
+} qudax_site_model;
+
+typedef struct {
+    int T_loc, t0;               /* local extent and first global timeslice */
+    int rank_fwd, rank_back;     /* T-ring neighbours */
+    long V_loc, V_h, V_s, face_sites; /* local volume, per-parity volume, XYZ, XYZ/2 */
+    int applies_bc_fwd, applies_bc_back; /* this rank owns global t=T-1 / t=0 */
+    size_t face_bytes[3];        /* one projected face (12 reals per site) in half/single/double,
+                                    half including its per-site norms */
+} qudax_partition;
+
+/* ---- host-only helpers (no GPU needed) ---- */
+int qudax_abi_version(void);
+const char *qudax_status_string(int status);
+/* Partition bookkeeping of rank `rank` of `nranks`. */
+qudax_status qudax_partition_info(const int global_dims[4], int nranks, int rank, qudax_partition *out);
+/* Site model for one Dslash kernel of `kind` (flops: 1320 + 504 clover + 48 xpay, Q16), or for
+ * the whole Mhat when kind = -1 (3696 flops / 2976 bytes at fp32 recon 12). */
+qudax_status qudax_model(int prec, int recon, int kind, qudax_site_model *out);
+/* ncclGetUniqueId into out[128] (rank 0 calls, caller broadcasts). */
+qudax_status qudax_nccl_unique_id(void *out128);
+
+/* ---- context ---- */
+qudax_status qudax_init(qudax_ctx **ctx, const qudax_init_param *p);
+qudax_status qudax_finalize(qudax_ctx *ctx);
+const char *qudax_last_error(const qudax_ctx *ctx);
+qudax_status qudax_sync(qudax_ctx *ctx);
+/* Number of library kernels launched by this ctx so far (for launch accounting). */
+long long qudax_launch_count(const qudax_ctx *ctx);
+qudax_status qudax_get_partition(const qudax_ctx *ctx, qudax_partition *out);
+
+/* ---- gauge field and clover (setup) ----
+ * Uploads the host slab, exchanges the gauge ghost / clover halo timeslices with the T
+ * neighbours (once), builds A and T^{-1} in fp64 on the device and stores gauge + clover in
+ * the outer and sloppy (precision, reconstruct) formats.  Returns QUDAX_ERR_UNSUPPORTED for
+ * reconstruct 8 when some link has |u01|^2 + |u02|^2 < 1e-6. */
+qudax_status qudax_gauge_load(qudax_ctx *ctx, const double *host_gauge, const qudax_gauge_param *p);
+
+/* ---- spinor fields ---- */
+size_t qudax_spinor_bytes(const qudax_ctx *ctx, int prec);
+/* Host full local slab (DeGrand-Rossi, fp64) -> one parity of a device field in `prec`.
+ * Basis change to the non-relativistic basis, parity split and precision conversion run in a
+ * device kernel; only the H2D copy is done by the host. */
+qudax_status qudax_spinor_load(qudax_ctx *ctx, void *dst, int prec, int parity, const double *host_src);
+/* Same, source already on the device (double[T_loc][Z][Y][X][4][3][2]). */
+qudax_status qudax_spinor_load_dev(qudax_ctx *ctx, void *dst, int prec, int parity, const double *dev_src);
+/* Device field (one parity) -> the sites of that parity of a host full local slab (DR basis,
+ * fp64).  Sites of the other parity are left untouched. */
+qudax_status qudax_spinor_store(qudax_ctx *ctx, double *host_dst, const void *src, int prec, int parity);
+qudax_status qudax_spinor_store_dev(qudax_ctx *ctx, double *dev_dst, const void *src, int prec, int parity);
+/* Precision conversion between two device parity fields (re-quantises half). */
+qudax_status qudax_spinor_convert(qudax_ctx *ctx, void *dst, int dst_prec, const void *src, int src_prec);
+
+/* ---- operator (stream-ordered) ---- */
+/* One Dslash kernel (with its halo exchange when partitioned): see qudax_dslash_kind.
+ * x is read only for CLOVER_XPAY (same parity as out). dagger: D -> D^dag = gamma5 D gamma5. */
+qudax_status qudax_dslash(qudax_ctx *ctx, void *out, const void *in, const void *x, int prec,
+                          int out_parity, int dagger, int kind, double a);
+/* out_e = Mhat in_e (dagger = 0) or Mhat^dag in_e (dagger = 1); 2 Dslash kernels + 2 halos. */
+qudax_status qudax_matpc(qudax_ctx *ctx, void *out, const void *in, int prec, int dagger);
+/* out_e = Mhat^dag Mhat in_e (the CGNR normal operator). */
+qudax_status qudax_mdagm(qudax_ctx *ctx, void *out, const void *in, int prec);
+
+/* ---- global reductions over the even (parity) field, fp64 accumulation, all ranks ---- */
+qudax_status qudax_norm2(qudax_ctx *ctx, const void *f, int prec, double *out);
+qudax_status qudax_cdot(qudax_ctx *ctx, const void *a, const void *b, int prec, double out_re_im[2]);
+
+/* ---- solver: mixed-precision reliable-update BiCGstab ---- */
+/* Host buffers: full local slabs (DR basis, fp64).  H2D of b and D2H of x are inside. */
+qudax_status qudax_solve_bicgstab(qudax_ctx *ctx, double *host_x, const double *host_b,
+                                  const qudax_solve_param *p, qudax_solve_stats *st);
+/* Same with device-resident fp64 full local slabs. */
+qudax_status qudax_solve_bicgstab_dev(qudax_ctx *ctx, double *dev_x, const double *dev_b,
+                                      const qudax_solve_param *p, qudax_solve_stats *st);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* QUDAX_H */

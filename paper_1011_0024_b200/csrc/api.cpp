@@ -1,0 +1,712 @@
+// api.cpp — the extern "C" boundary (include/qudax.h) and the host runtime behind it:
+// context, device memory, gauge/clover setup, the T-direction halo orchestration
+// (pack -> NCCL send/recv on a comm stream -> interior kernel -> boundary kernel,
+// P:692-720), and global reductions.
+#include <cuda_runtime.h>
+#include <nccl.h>
+
+#include <algorithm>
+#include <chrono>
+#include <cmath>
+#include <cstring>
+
+#include "ctx.h"
+
+using qx::Error;
+
+#define QX_NCCL(call)                                                                              \
+    do {                                                                                           \
+        ncclResult_t r_ = (call);                                                                  \
+        if (r_ != ncclSuccess) throw Error(QUDAX_ERR_NCCL, std::string(#call) + ": " + ncclGetErrorString(r_)); \
+    } while (0)
+
+namespace qx {
+
+void *dalloc(qudax_ctx *c, size_t bytes) {
+    if (bytes == 0) bytes = 16;
+    void *p = nullptr;
+    if (c->dev_alloc) {
+        p = c->dev_alloc(bytes, c->alloc_user);
+        if (!p) throw Error(QUDAX_ERR_OOM, "dev_alloc hook returned NULL for " + std::to_string(bytes) + " bytes");
+    } else {
+        cudaError_t e = cudaMalloc(&p, bytes);
+        if (e != cudaSuccess) {
+            cudaGetLastError();
+            throw Error(QUDAX_ERR_OOM, "cudaMalloc(" + std::to_string(bytes) + "): " + cudaGetErrorString(e));
+        }
+    }
+    c->allocs.push_back(p);
+    return p;
+}
+
+void *halloc(qudax_ctx *c, size_t bytes) {
+    void *p = nullptr;
+    QX_CUDA(cudaMallocHost(&p, std::max<size_t>(bytes, 16)));
+    c->host_allocs.push_back(p);
+    return p;
+}
+
+static void dfree(qudax_ctx *c, void *p) {
+    if (!p) return;
+    auto it = std::find(c->allocs.begin(), c->allocs.end(), p);
+    if (it != c->allocs.end()) c->allocs.erase(it);
+    if (c->dev_free) c->dev_free(p, c->alloc_user);
+    else cudaFree(p);
+}
+
+void check_prec(int prec) {
+    QX_CHECK(prec == 2 || prec == 4 || prec == 8, QUDAX_ERR_ARG, "precision must be 2, 4 or 8");
+}
+
+static qudax_ctx::GaugeCopy &gauge_for(qudax_ctx *c, int prec) {
+    QX_CHECK(c->gauge_loaded, QUDAX_ERR_STATE, "gauge field not loaded");
+    for (int k = 0; k < c->ncopies; ++k)
+        if (c->gcopy[k].prec == prec) return c->gcopy[k];
+    throw Error(QUDAX_ERR_ARG, "no gauge copy in precision " + std::to_string(prec));
+}
+
+static qudax_ctx::Halo &halo_for(qudax_ctx *c, int prec) {
+    auto &h = c->halo[prec_idx(prec)];
+    if (!h.valid) {
+        h.bytes = face_bytes(prec, c->g.fstride);
+        h.sb = dalloc(c, h.bytes);
+        h.sf = dalloc(c, h.bytes);
+        h.gb = dalloc(c, h.bytes);
+        h.gf = dalloc(c, h.bytes);
+        if (c->comm == QUDAX_COMM_HOST) {
+            h.h_sb = halloc(c, h.bytes);
+            h.h_sf = halloc(c, h.bytes);
+            h.h_gb = halloc(c, h.bytes);
+            h.h_gf = halloc(c, h.bytes);
+        }
+        h.valid = true;
+    }
+    return h;
+}
+
+static inline int rank_fwd(const Geom &g) { return (g.rank + 1) % g.nranks; }
+static inline int rank_back(const Geom &g) { return (g.rank - 1 + g.nranks) % g.nranks; }
+
+// Exchange of two device buffers of `bytes` with the T neighbours: send_fwd -> rank+1,
+// send_back -> rank-1, recv_back <- rank-1, recv_fwd <- rank+1.  On NCCL it is enqueued on
+// `s`; on HOST it is staged through pinned memory and completes before return.
+static void exchange(qudax_ctx *c, const void *send_fwd, const void *send_back, void *recv_back, void *recv_fwd,
+                     size_t bytes, cudaStream_t s, void *h_sf, void *h_sb, void *h_gb, void *h_gf) {
+    const Geom &g = c->g;
+    if (c->comm == QUDAX_COMM_NCCL) {
+        QX_NCCL(ncclGroupStart());
+        QX_NCCL(ncclSend(send_fwd, bytes, ncclChar, rank_fwd(g), c->nccl, s));
+        QX_NCCL(ncclRecv(recv_back, bytes, ncclChar, rank_back(g), c->nccl, s));
+        QX_NCCL(ncclSend(send_back, bytes, ncclChar, rank_back(g), c->nccl, s));
+        QX_NCCL(ncclRecv(recv_fwd, bytes, ncclChar, rank_fwd(g), c->nccl, s));
+        QX_NCCL(ncclGroupEnd());
+    } else if (c->comm == QUDAX_COMM_HOST) {
+        QX_CUDA(cudaMemcpyAsync(h_sf, send_fwd, bytes, cudaMemcpyDeviceToHost, s));
+        QX_CUDA(cudaMemcpyAsync(h_sb, send_back, bytes, cudaMemcpyDeviceToHost, s));
+        QX_CUDA(cudaStreamSynchronize(s));
+        int rc = c->host_exchange(h_sf, h_sb, h_gb, h_gf, bytes, c->comm_user);
+        if (rc) throw Error(QUDAX_ERR_COMM, "host_exchange hook failed");
+        QX_CUDA(cudaMemcpyAsync(recv_back, h_gb, bytes, cudaMemcpyHostToDevice, s));
+        QX_CUDA(cudaMemcpyAsync(recv_fwd, h_gf, bytes, cudaMemcpyHostToDevice, s));
+    } else {
+        throw Error(QUDAX_ERR_STATE, "exchange without a transport");
+    }
+}
+
+static void launch_dslash_any(int prec, int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
+    if (prec == 8) launch_dslash_f64(recon, dagger, kind, a, s);
+    else if (prec == 4) launch_dslash_f32(recon, dagger, kind, a, s);
+    else launch_dslash_f16(recon, dagger, kind, a, s);
+    QX_CUDA(cudaGetLastError());
+}
+
+void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
+               double a) {
+    check_prec(prec);
+    QX_CHECK(p == 0 || p == 1, QUDAX_ERR_ARG, "parity must be 0 or 1");
+    QX_CHECK(kind >= 0 && kind <= 2, QUDAX_ERR_ARG, "bad dslash kind");
+    QX_CHECK(out && in && (kind != QUDAX_CLOVER_XPAY || x), QUDAX_ERR_ARG, "null field");
+    QX_CHECK(out != in, QUDAX_ERR_ARG, "dslash cannot run in place");
+    auto &gc = gauge_for(c, prec);
+    const Geom &g = c->g;
+    DslashArgs args{};
+    args.X = g.X; args.Y = g.Y; args.Z = g.Z; args.T_loc = g.T_loc; args.Xh = g.Xh;
+    args.Vh = (int)g.Vh; args.F = (int)g.F;
+    args.stride = g.stride; args.fstride = g.fstride;
+    args.parity = p;
+    args.bc_fwd = (g.rank == g.nranks - 1) ? (double)c->t_bc : 1.0;
+    args.bc_back = (g.rank == 0) ? (double)c->t_bc : 1.0;
+    args.a = a;
+    args.in = in; args.out = out; args.x = x;
+    for (int m = 0; m < 4; ++m)
+        for (int q = 0; q < 2; ++q) args.gauge[m][q] = gc.d[m][q];
+    args.gauge_ghost = gc.ghost[1 - p];
+    if (kind != QUDAX_HOP) {
+        auto &cl = c->clov[prec_idx(prec)];
+        QX_CHECK(cl.valid, QUDAX_ERR_STATE, "no clover in this precision");
+        args.clover = (kind == QUDAX_CLOVER_XPAY) ? cl.T[p] : cl.Tinv[p];
+    }
+    if (c->comm == QUDAX_COMM_NONE) {
+        args.ghosted = 0;
+        args.range = RANGE_ALL;
+        args.nthreads = (int)g.Vh;
+        launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+        c->launches += 1;
+        return;
+    }
+    auto &h = halo_for(c, prec);
+    args.ghosted = 1;
+    args.ghost_back = h.gb;
+    args.ghost_fwd = h.gf;
+    if (c->comm == QUDAX_COMM_NCCL) {
+        // comm stream: wait for `in` (and for the previous boundary kernel, which read the ghosts)
+        QX_CUDA(cudaEventRecord(c->ev_in, c->stream));
+        QX_CUDA(cudaStreamWaitEvent(c->comm_stream, c->ev_in, 0));
+        launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, c->comm_stream);
+        exchange(c, h.sf, h.sb, h.gb, h.gf, h.bytes, c->comm_stream, nullptr, nullptr, nullptr, nullptr);
+        QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
+        c->launches += 1;
+        if (c->overlap && g.T_loc > 2) {
+            args.range = RANGE_INTERIOR;
+            args.nthreads = (int)((g.T_loc - 2) * g.F);
+            launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+            QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
+            args.range = RANGE_BOUNDARY;
+            args.nthreads = (int)(2 * g.F);
+            launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+            c->launches += 2;
+        } else {
+            QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
+            args.range = RANGE_ALL;
+            args.nthreads = (int)g.Vh;
+            launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+            c->launches += 1;
+        }
+    } else {  // HOST: paper strategy 1 (no overlap)
+        launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, c->stream);
+        exchange(c, h.sf, h.sb, h.gb, h.gf, h.bytes, c->stream, h.h_sf, h.h_sb, h.h_gb, h.h_gf);
+        args.range = RANGE_ALL;
+        args.nthreads = (int)g.Vh;
+        launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+        c->launches += 2;
+    }
+}
+
+static void *tmp_odd(qudax_ctx *c, int prec) {
+    auto &t = c->tmp_odd[prec_idx(prec)];
+    if (!t) t = dalloc(c, spinor_bytes(prec, c->g.stride));
+    return t;
+}
+static void *tmp_even(qudax_ctx *c, int prec) {
+    auto &t = c->tmp_even[prec_idx(prec)];
+    if (!t) t = dalloc(c, spinor_bytes(prec, c->g.stride));
+    return t;
+}
+
+// Mhat = T_ee - kappa^2 D_eo T_oo^{-1} D_oe (asymmetric Schur form on even sites)
+void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger) {
+    void *t = tmp_odd(c, prec);
+    dslash_op(c, t, in, nullptr, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0);
+    dslash_op(c, out, t, in, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa);
+}
+
+void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int parity, bool inverse) {
+    auto &cl = c->clov[prec_idx(prec)];
+    QX_CHECK(cl.valid, QUDAX_ERR_STATE, "no clover in this precision");
+    launch_clover_apply(prec, c->g, inverse ? cl.Tinv[parity] : cl.T[parity], in, out, c->stream);
+    c->launches += 1;
+}
+
+static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res) {
+    if (c->g.nranks > 1 && c->comm == QUDAX_COMM_NCCL) {
+        QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl, c->stream));
+    }
+    QX_CUDA(cudaMemcpyAsync(c->h_red, dev_vals, sizeof(double) * n, cudaMemcpyDeviceToHost, c->stream));
+    QX_CUDA(cudaStreamSynchronize(c->stream));
+    if (c->g.nranks > 1 && c->comm == QUDAX_COMM_HOST) {
+        if (c->host_allreduce(c->h_red, n, c->comm_user)) throw Error(QUDAX_ERR_COMM, "host_allreduce hook failed");
+    }
+    for (int k = 0; k < n; ++k) res[k] = c->h_red[k];
+}
+
+int blas_op(qudax_ctx *c, int op, int prec, void *const *f, const double *coef, double *res) {
+    int n = blas_run(op, prec, c->g, f, coef, c->partials, c->red_out, c->stream);
+    c->launches += 1 + (n ? 1 : 0);
+    if (n) global_sum(c, c->red_out, n, res);
+    return n;
+}
+
+void xpy_mixed_op(qudax_ctx *c, int pd, int ps, const void *x, void *y) {
+    blas_xpy_mixed(pd, ps, c->g, x, y, c->stream);
+    c->launches += 1;
+}
+
+void convert_op(qudax_ctx *c, void *dst, int pd, const void *src, int ps) {
+    launch_spinor_convert(pd, ps, c->g, dst, src, c->stream);
+    c->launches += 1;
+}
+
+static void gauge_load(qudax_ctx *c, const double *host, const qudax_gauge_param *p) {
+    QX_CHECK(host && p, QUDAX_ERR_ARG, "null gauge or param");
+    const Geom &g = c->g;
+    for (int k = 0; k < 2; ++k) {
+        int pr = k ? p->prec_sloppy : p->prec, rc = k ? p->recon_sloppy : p->recon;
+        check_prec(pr);
+        QX_CHECK(rc == 18 || rc == 12 || rc == 8, QUDAX_ERR_ARG, "recon must be 18, 12 or 8");
+    }
+    QX_CHECK(p->t_boundary == 1 || p->t_boundary == -1, QUDAX_ERR_ARG, "t_boundary must be +1 or -1");
+    // drop a previous configuration's copies (fields of the previous load are released)
+    for (int k = 0; k < c->ncopies; ++k) {
+        for (int m = 0; m < 4; ++m)
+            for (int q = 0; q < 2; ++q) dfree(c, c->gcopy[k].d[m][q]);
+        dfree(c, c->gcopy[k].ghost[0]);
+        dfree(c, c->gcopy[k].ghost[1]);
+        c->gcopy[k] = qudax_ctx::GaugeCopy{};
+    }
+    for (auto &cl : c->clov) {
+        if (!cl.valid) continue;
+        for (int q = 0; q < 2; ++q) { dfree(c, cl.T[q]); dfree(c, cl.Tinv[q]); }
+        cl = qudax_ctx::Clover{};
+    }
+    c->ncopies = 0;
+    c->gauge_loaded = false;
+    c->kappa = p->kappa;
+    c->csw = p->csw;
+    c->t_bc = p->t_boundary;
+
+    // 1. upload the slab into the extended fp64 buffer [T_loc+2][4][Vs][18]
+    const size_t link_d = 18;
+    const size_t slice = (size_t)4 * g.Vs * link_d;  // doubles per extended timeslice
+    double *ext = static_cast<double *>(dalloc(c, sizeof(double) * slice * (g.T_loc + 2)));
+    for (int mu = 0; mu < 4; ++mu) {
+        QX_CUDA(cudaMemcpy2DAsync(ext + slice + (size_t)mu * g.Vs * link_d, sizeof(double) * slice,
+                                  host + (size_t)mu * g.T_loc * g.Vs * link_d, sizeof(double) * g.Vs * link_d,
+                                  sizeof(double) * g.Vs * link_d, g.T_loc, cudaMemcpyHostToDevice, c->stream));
+    }
+    // 2. gauge ghost + clover halo: one full timeslice from each T neighbour, once
+    double *first = ext + slice, *last = ext + slice * g.T_loc;
+    double *halo_back = ext, *halo_fwd = ext + slice * (g.T_loc + 1);
+    if (c->comm == QUDAX_COMM_NONE || g.nranks == 1) {
+        QX_CUDA(cudaMemcpyAsync(halo_back, last, sizeof(double) * slice, cudaMemcpyDeviceToDevice, c->stream));
+        QX_CUDA(cudaMemcpyAsync(halo_fwd, first, sizeof(double) * slice, cudaMemcpyDeviceToDevice, c->stream));
+    } else {
+        void *hs[4] = {nullptr, nullptr, nullptr, nullptr};
+        if (c->comm == QUDAX_COMM_HOST)
+            for (auto &q : hs) q = halloc(c, sizeof(double) * slice);
+        exchange(c, last, first, halo_back, halo_fwd, sizeof(double) * slice, c->stream, hs[0], hs[1], hs[2], hs[3]);
+    }
+    // 3. pack each (precision, reconstruct) copy
+    int *bad = c->d_flag;
+    QX_CUDA(cudaMemsetAsync(bad, 0, sizeof(int), c->stream));
+    for (int k = 0; k < 2; ++k) {
+        int pr = k ? p->prec_sloppy : p->prec, rc = k ? p->recon_sloppy : p->recon;
+        if (k == 1 && pr == p->prec) break;  // sloppy == outer precision: one copy
+        auto &gc = c->gcopy[c->ncopies++];
+        gc.prec = pr;
+        gc.recon = rc;
+        const size_t b = soa_bytes(pr, rc, g.stride);
+        for (int m = 0; m < 4; ++m)
+            for (int q = 0; q < 2; ++q) gc.d[m][q] = dalloc(c, b);
+        for (int q = 0; q < 2; ++q) gc.ghost[q] = dalloc(c, soa_bytes(pr, rc, g.fstride));
+        launch_gauge_pack2(pr, rc, g, ext, gc.d, gc.ghost, bad, c->stream);
+        c->launches += 1;
+    }
+    // 4. clover T and T^{-1} in fp64, then each working precision
+    double *T64[2], *I64[2];
+    for (int q = 0; q < 2; ++q) {
+        T64[q] = static_cast<double *>(dalloc(c, sizeof(double) * 72 * g.Vh));
+        I64[q] = static_cast<double *>(dalloc(c, sizeof(double) * 72 * g.Vh));
+    }
+    int *bad_clover = c->d_flag + 1;
+    QX_CUDA(cudaMemsetAsync(bad_clover, 0, sizeof(int), c->stream));
+    launch_clover_build(g, ext, p->kappa, p->csw, T64, I64, bad_clover, c->stream);
+    c->launches += 1;
+    for (int k = 0; k < c->ncopies; ++k) {
+        int pr = c->gcopy[k].prec;
+        auto &cl = c->clov[prec_idx(pr)];
+        if (cl.valid) continue;
+        for (int q = 0; q < 2; ++q) {
+            cl.T[q] = dalloc(c, clover_bytes(pr, g.stride));
+            cl.Tinv[q] = dalloc(c, clover_bytes(pr, g.stride));
+            launch_clover_pack(pr, g, T64[q], cl.T[q], c->stream);
+            launch_clover_pack(pr, g, I64[q], cl.Tinv[q], c->stream);
+            c->launches += 2;
+        }
+        cl.valid = true;
+    }
+    int hbad[2];
+    QX_CUDA(cudaMemcpyAsync(hbad, c->d_flag, sizeof(hbad), cudaMemcpyDeviceToHost, c->stream));
+    QX_CUDA(cudaStreamSynchronize(c->stream));
+    for (int q = 0; q < 2; ++q) { dfree(c, T64[q]); dfree(c, I64[q]); }
+    dfree(c, ext);
+    QX_CHECK(hbad[1] == 0, QUDAX_ERR_ARG, "clover term singular on " + std::to_string(hbad[1]) + " chiral blocks");
+    bool r8 = (p->recon == 8) || (p->recon_sloppy == 8 && p->prec_sloppy != p->prec);
+    if (r8 && hbad[0]) {
+        throw Error(QUDAX_ERR_UNSUPPORTED, "reconstruct 8 rejected: " + std::to_string(hbad[0]) +
+                                               " links with |u01|^2+|u02|^2 < 1e-6 (e.g. unit gauge)");
+    }
+    c->gauge_loaded = true;
+}
+
+}  // namespace qx
+
+// ============================================================================ C ABI
+using namespace qx;
+
+namespace {
+template <typename F>
+qudax_status guard(qudax_ctx *c, F &&fn) {
+    if (c && c->sticky) return QUDAX_ERR_STATE;
+    try {
+        fn();
+        return QUDAX_OK;
+    } catch (const Error &e) {
+        if (c) {
+            c->err = e.what();
+            if (e.status == QUDAX_ERR_CUDA || e.status == QUDAX_ERR_NCCL) c->sticky = true;
+        }
+        return e.status;
+    } catch (const std::exception &e) {
+        if (c) c->err = e.what();
+        return QUDAX_ERR_STATE;
+    } catch (...) {
+        if (c) c->err = "unknown exception";
+        return QUDAX_ERR_STATE;
+    }
+}
+
+qudax_status fill_partition(const int gd[4], int nranks, int rank, qudax_partition *o) {
+    if (!gd || !o || nranks < 1 || rank < 0 || rank >= nranks) return QUDAX_ERR_ARG;
+    for (int k = 0; k < 4; ++k)
+        if (gd[k] < 1) return QUDAX_ERR_ARG;
+    if (gd[0] % 2) return QUDAX_ERR_ARG;
+    if (gd[3] % nranks) return QUDAX_ERR_ARG;
+    const int T_loc = gd[3] / nranks;
+    if (T_loc < 2 || T_loc % 2) return QUDAX_ERR_ARG;
+    std::memset(o, 0, sizeof(*o));
+    o->T_loc = T_loc;
+    o->t0 = rank * T_loc;
+    o->rank_fwd = (rank + 1) % nranks;
+    o->rank_back = (rank - 1 + nranks) % nranks;
+    o->V_s = (long)gd[0] * gd[1] * gd[2];
+    o->V_loc = o->V_s * T_loc;
+    o->V_h = o->V_loc / 2;
+    o->face_sites = o->V_s / 2;
+    o->applies_bc_fwd = (rank == nranks - 1);
+    o->applies_bc_back = (rank == 0);
+    o->face_bytes[0] = (size_t)o->face_sites * (12 * 2 + 4);
+    o->face_bytes[1] = (size_t)o->face_sites * 12 * 4;
+    o->face_bytes[2] = (size_t)o->face_sites * 12 * 8;
+    return QUDAX_OK;
+}
+}  // namespace
+
+extern "C" {
+
+int qudax_abi_version(void) { return QUDAX_ABI_VERSION; }
+
+const char *qudax_status_string(int s) {
+    switch (s) {
+        case QUDAX_OK: return "ok";
+        case QUDAX_ERR_ARG: return "invalid argument";
+        case QUDAX_ERR_STATE: return "invalid state";
+        case QUDAX_ERR_CUDA: return "CUDA error";
+        case QUDAX_ERR_NCCL: return "NCCL error";
+        case QUDAX_ERR_UNSUPPORTED: return "unsupported";
+        case QUDAX_ERR_NOT_CONVERGED: return "not converged";
+        case QUDAX_ERR_OOM: return "out of device memory";
+        case QUDAX_ERR_COMM: return "host transport failed";
+        default: return "unknown status";
+    }
+}
+
+qudax_status qudax_partition_info(const int global_dims[4], int nranks, int rank, qudax_partition *out) {
+    return fill_partition(global_dims, nranks, rank, out);
+}
+
+qudax_status qudax_model(int prec, int recon, int kind, qudax_site_model *o) {
+    if (!o || (prec != 2 && prec != 4 && prec != 8) || (recon != 18 && recon != 12 && recon != 8) || kind < -1 ||
+        kind > 2)
+        return QUDAX_ERR_ARG;
+    const double w = prec;
+    const double norm = (prec == 2) ? 4 : 0;
+    const double sp = 24 * w + norm, hsp = 12 * w + norm, link = recon * w, clov = 72 * w + (prec == 2 ? 8 : 0);
+    auto one = [&](int k, qudax_site_model *m) {
+        const double cl = (k == QUDAX_HOP) ? 0 : clov;
+        const double xs = (k == QUDAX_CLOVER_XPAY) ? sp : 0;
+        m->flops = 1320 + (k == QUDAX_HOP ? 0 : 504) + (k == QUDAX_CLOVER_XPAY ? 48 : 0);
+        m->bytes_paper = 6 * sp + 2 * hsp + 8 * link + cl + xs + sp;
+        m->bytes_compulsory = 8 * link + sp + cl + xs + sp;
+    };
+    if (kind >= 0) {
+        one(kind, o);
+    } else {
+        qudax_site_model a, b;
+        one(QUDAX_CLOVER_INV, &a);
+        one(QUDAX_CLOVER_XPAY, &b);
+        o->flops = a.flops + b.flops;
+        o->bytes_paper = a.bytes_paper + b.bytes_paper;
+        o->bytes_compulsory = a.bytes_compulsory + b.bytes_compulsory;
+    }
+    return QUDAX_OK;
+}
+
+qudax_status qudax_nccl_unique_id(void *out128) {
+    if (!out128) return QUDAX_ERR_ARG;
+    ncclUniqueId id;
+    if (ncclGetUniqueId(&id) != ncclSuccess) return QUDAX_ERR_NCCL;
+    static_assert(sizeof(id) == 128, "ncclUniqueId size");
+    std::memcpy(out128, &id, 128);
+    return QUDAX_OK;
+}
+
+qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
+    if (!out || !p) return QUDAX_ERR_ARG;
+    *out = nullptr;
+    qudax_partition part;
+    if (fill_partition(p->global_dims, p->nranks, p->rank, &part) != QUDAX_OK) return QUDAX_ERR_ARG;
+    if (p->comm == QUDAX_COMM_NONE && p->nranks != 1) return QUDAX_ERR_ARG;
+    if (p->comm == QUDAX_COMM_NCCL && !p->nccl_id) return QUDAX_ERR_ARG;
+    if (p->comm == QUDAX_COMM_HOST && (!p->host_exchange || !p->host_allreduce)) return QUDAX_ERR_ARG;
+    if (p->comm < 0 || p->comm > 2) return QUDAX_ERR_ARG;
+    auto *c = new qudax_ctx();
+    qudax_status st = guard(c, [&] {
+        Geom &g = c->g;
+        g.X = p->global_dims[0]; g.Y = p->global_dims[1]; g.Z = p->global_dims[2]; g.T = p->global_dims[3];
+        g.nranks = p->nranks; g.rank = p->rank;
+        g.T_loc = part.T_loc; g.t0 = part.t0;
+        g.Xh = g.X / 2;
+        g.Vs = part.V_s; g.V = part.V_loc; g.Vh = part.V_h; g.F = part.face_sites;
+        g.stride = pad64(g.Vh);
+        g.fstride = pad64(g.F);
+        QX_CHECK(g.V < (1L << 30), QUDAX_ERR_ARG, "local volume too large for 32-bit site indexing");
+        c->device = p->device;
+        c->comm = p->comm;
+        c->overlap = p->overlap;
+        c->dev_alloc = p->dev_alloc; c->dev_free = p->dev_free; c->alloc_user = p->alloc_user;
+        c->host_exchange = p->host_exchange; c->host_allreduce = p->host_allreduce; c->comm_user = p->comm_user;
+        QX_CUDA(cudaSetDevice(p->device));
+        if (p->stream) {
+            c->stream = reinterpret_cast<cudaStream_t>(p->stream);
+        } else {
+            QX_CUDA(cudaStreamCreateWithFlags(&c->stream, cudaStreamNonBlocking));
+            c->own_stream = true;
+        }
+        int lo, hi;
+        QX_CUDA(cudaDeviceGetStreamPriorityRange(&lo, &hi));
+        QX_CUDA(cudaStreamCreateWithPriority(&c->comm_stream, cudaStreamNonBlocking, hi));
+        QX_CUDA(cudaEventCreateWithFlags(&c->ev_in, cudaEventDisableTiming));
+        QX_CUDA(cudaEventCreateWithFlags(&c->ev_halo, cudaEventDisableTiming));
+        if (c->comm == QUDAX_COMM_NCCL) {
+            ncclUniqueId id;
+            std::memcpy(&id, p->nccl_id, sizeof(id));
+            QX_NCCL(ncclCommInitRank(&c->nccl, g.nranks, id, g.rank));
+        }
+        c->partials = static_cast<double *>(dalloc(c, sizeof(double) * 4 * blas_partial_blocks()));
+        c->red_out = static_cast<double *>(dalloc(c, sizeof(double) * 8));
+        c->h_red = static_cast<double *>(halloc(c, sizeof(double) * 8));
+        c->d_flag = static_cast<int *>(dalloc(c, sizeof(int) * 4));
+    });
+    if (st != QUDAX_OK) {
+        qudax_finalize(c);
+        return st;
+    }
+    *out = c;
+    return QUDAX_OK;
+}
+
+qudax_status qudax_finalize(qudax_ctx *c) {
+    if (!c) return QUDAX_ERR_ARG;
+    if (c->stream) cudaStreamSynchronize(c->stream);
+    if (c->comm_stream) cudaStreamSynchronize(c->comm_stream);
+    if (c->nccl) ncclCommDestroy(c->nccl);
+    for (void *p : c->allocs) {
+        if (c->dev_free) c->dev_free(p, c->alloc_user);
+        else cudaFree(p);
+    }
+    for (void *p : c->host_allocs) cudaFreeHost(p);
+    if (c->ev_in) cudaEventDestroy(c->ev_in);
+    if (c->ev_halo) cudaEventDestroy(c->ev_halo);
+    if (c->comm_stream) cudaStreamDestroy(c->comm_stream);
+    if (c->own_stream && c->stream) cudaStreamDestroy(c->stream);
+    delete c;
+    return QUDAX_OK;
+}
+
+const char *qudax_last_error(const qudax_ctx *c) { return c ? c->err.c_str() : "null context"; }
+
+qudax_status qudax_sync(qudax_ctx *c) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        QX_CUDA(cudaStreamSynchronize(c->comm_stream));
+    });
+}
+
+long long qudax_launch_count(const qudax_ctx *c) { return c ? c->launches : -1; }
+
+qudax_status qudax_get_partition(const qudax_ctx *c, qudax_partition *out) {
+    if (!c || !out) return QUDAX_ERR_ARG;
+    const int gd[4] = {c->g.X, c->g.Y, c->g.Z, c->g.T};
+    return fill_partition(gd, c->g.nranks, c->g.rank, out);
+}
+
+qudax_status qudax_gauge_load(qudax_ctx *c, const double *host_gauge, const qudax_gauge_param *p) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] { gauge_load(c, host_gauge, p); });
+}
+
+size_t qudax_spinor_bytes(const qudax_ctx *c, int prec) {
+    if (!c || (prec != 2 && prec != 4 && prec != 8)) return 0;
+    return spinor_bytes(prec, c->g.stride);
+}
+
+static double *stage_buf(qudax_ctx *c) {
+    if (!c->stage) c->stage = static_cast<double *>(dalloc(c, sizeof(double) * 24 * c->g.V));
+    return c->stage;
+}
+
+qudax_status qudax_spinor_load(qudax_ctx *c, void *dst, int prec, int parity, const double *host_src) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        check_prec(prec);
+        QX_CHECK(dst && host_src && (parity == 0 || parity == 1), QUDAX_ERR_ARG, "spinor_load: bad argument");
+        double *st = stage_buf(c);
+        QX_CUDA(cudaMemcpyAsync(st, host_src, sizeof(double) * 24 * c->g.V, cudaMemcpyHostToDevice, c->stream));
+        launch_spinor_import(prec, c->g, parity, st, dst, c->stream);
+        c->launches += 1;
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+    });
+}
+
+qudax_status qudax_spinor_load_dev(qudax_ctx *c, void *dst, int prec, int parity, const double *dev_src) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        check_prec(prec);
+        QX_CHECK(dst && dev_src && (parity == 0 || parity == 1), QUDAX_ERR_ARG, "spinor_load_dev: bad argument");
+        launch_spinor_import(prec, c->g, parity, dev_src, dst, c->stream);
+        c->launches += 1;
+    });
+}
+
+qudax_status qudax_spinor_store(qudax_ctx *c, double *host_dst, const void *src, int prec, int parity) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        check_prec(prec);
+        QX_CHECK(src && host_dst && (parity == 0 || parity == 1), QUDAX_ERR_ARG, "spinor_store: bad argument");
+        double *st = stage_buf(c);
+        const size_t n = sizeof(double) * 24 * c->g.V;
+        QX_CUDA(cudaMemcpyAsync(st, host_dst, n, cudaMemcpyHostToDevice, c->stream));  // keep other parity
+        launch_spinor_export(prec, c->g, parity, src, st, c->stream);
+        c->launches += 1;
+        QX_CUDA(cudaMemcpyAsync(host_dst, st, n, cudaMemcpyDeviceToHost, c->stream));
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+    });
+}
+
+qudax_status qudax_spinor_store_dev(qudax_ctx *c, double *dev_dst, const void *src, int prec, int parity) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        check_prec(prec);
+        QX_CHECK(src && dev_dst && (parity == 0 || parity == 1), QUDAX_ERR_ARG, "spinor_store_dev: bad argument");
+        launch_spinor_export(prec, c->g, parity, src, dev_dst, c->stream);
+        c->launches += 1;
+    });
+}
+
+qudax_status qudax_spinor_convert(qudax_ctx *c, void *dst, int dst_prec, const void *src, int src_prec) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        check_prec(dst_prec);
+        check_prec(src_prec);
+        QX_CHECK(dst && src && dst != src, QUDAX_ERR_ARG, "spinor_convert: bad argument");
+        convert_op(c, dst, dst_prec, src, src_prec);
+    });
+}
+
+qudax_status qudax_dslash(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int out_parity,
+                          int dagger, int kind, double a) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] { dslash_op(c, out, in, x, prec, out_parity, dagger ? 1 : 0, kind, a); });
+}
+
+qudax_status qudax_matpc(qudax_ctx *c, void *out, const void *in, int prec, int dagger) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        QX_CHECK(out && in && out != in, QUDAX_ERR_ARG, "matpc: bad fields");
+        matpc_op(c, out, in, prec, dagger ? 1 : 0);
+    });
+}
+
+qudax_status qudax_mdagm(qudax_ctx *c, void *out, const void *in, int prec) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        QX_CHECK(out && in && out != in, QUDAX_ERR_ARG, "mdagm: bad fields");
+        check_prec(prec);
+        void *t = tmp_even(c, prec);
+        matpc_op(c, t, in, prec, 0);
+        matpc_op(c, out, t, prec, 1);
+    });
+}
+
+qudax_status qudax_norm2(qudax_ctx *c, const void *f, int prec, double *out) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        check_prec(prec);
+        QX_CHECK(f && out, QUDAX_ERR_ARG, "norm2: null");
+        void *fs[1] = {const_cast<void *>(f)};
+        blas_op(c, OP_NORM2, prec, fs, nullptr, out);
+    });
+}
+
+qudax_status qudax_cdot(qudax_ctx *c, const void *a, const void *b, int prec, double out[2]) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        check_prec(prec);
+        QX_CHECK(a && b && out, QUDAX_ERR_ARG, "cdot: null");
+        void *fs[2] = {const_cast<void *>(a), const_cast<void *>(b)};
+        blas_op(c, OP_CDOT, prec, fs, nullptr, out);
+    });
+}
+
+qudax_status qudax_solve_bicgstab_dev(qudax_ctx *c, double *x, const double *b, const qudax_solve_param *p,
+                                      qudax_solve_stats *st) {
+    if (!c) return QUDAX_ERR_ARG;
+    qudax_status s = guard(c, [&] {
+        QX_CHECK(x && b && p && st, QUDAX_ERR_ARG, "solve: null argument");
+        auto t0 = std::chrono::steady_clock::now();
+        solve_dev(c, x, b, p, st);
+        st->secs = std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
+        st->gflops = st->flops / st->secs * 1e-9;
+    });
+    if (s == QUDAX_OK && st && p && p->tol > 0 && st->true_res > p->tol * (1 + 1e-3)) return QUDAX_ERR_NOT_CONVERGED;
+    return s;
+}
+
+qudax_status qudax_solve_bicgstab(qudax_ctx *c, double *host_x, const double *host_b, const qudax_solve_param *p,
+                                  qudax_solve_stats *st) {
+    if (!c) return QUDAX_ERR_ARG;
+    double *db = nullptr, *dx = nullptr;
+    auto t0 = std::chrono::steady_clock::now();
+    qudax_status s = guard(c, [&] {
+        QX_CHECK(host_x && host_b && p && st, QUDAX_ERR_ARG, "solve: null argument");
+        const size_t n = sizeof(double) * 24 * c->g.V;
+        db = static_cast<double *>(dalloc(c, n));
+        dx = static_cast<double *>(dalloc(c, n));
+        QX_CUDA(cudaMemcpyAsync(db, host_b, n, cudaMemcpyHostToDevice, c->stream));
+        solve_dev(c, dx, db, p, st);
+        QX_CUDA(cudaMemcpyAsync(host_x, dx, n, cudaMemcpyDeviceToHost, c->stream));
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        dfree(c, db);
+        dfree(c, dx);
+        db = dx = nullptr;
+        st->secs = std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
+        st->gflops = st->flops / st->secs * 1e-9;
+    });
+    if (db) { cudaStreamSynchronize(c->stream); dfree(c, db); }
+    if (dx) dfree(c, dx);
+    if (s == QUDAX_OK && p->tol > 0 && st->true_res > p->tol * (1 + 1e-3)) return QUDAX_ERR_NOT_CONVERGED;
+    return s;
+}
+
+}  // extern "C"

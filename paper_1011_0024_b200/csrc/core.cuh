@@ -1,0 +1,293 @@
+// core.cuh — device building blocks: complex arithmetic, site-major SoA storage in the three
+// precisions (P:396-424 field ordering; P:507-520 half = 16-bit fixed point with a per-site
+// norm), SU(3) link reconstruction (P:475-478 two-row; reading Q6 eight-parameter).
+#pragma once
+#include <cuda_runtime.h>
+#include <cstdint>
+
+namespace qx {
+
+template <typename R>
+struct Cx {
+    R r, i;
+};
+template <typename R> __device__ __forceinline__ Cx<R> cx(R r, R i) { return Cx<R>{r, i}; }
+template <typename R> __device__ __forceinline__ Cx<R> operator+(Cx<R> a, Cx<R> b) { return {a.r + b.r, a.i + b.i}; }
+template <typename R> __device__ __forceinline__ Cx<R> operator-(Cx<R> a, Cx<R> b) { return {a.r - b.r, a.i - b.i}; }
+template <typename R> __device__ __forceinline__ Cx<R> operator*(Cx<R> a, Cx<R> b) {
+    return {a.r * b.r - a.i * b.i, a.r * b.i + a.i * b.r};
+}
+template <typename R> __device__ __forceinline__ Cx<R> operator*(R s, Cx<R> a) { return {s * a.r, s * a.i}; }
+template <typename R> __device__ __forceinline__ Cx<R> conj(Cx<R> a) { return {a.r, -a.i}; }
+// a * conj(b)
+template <typename R> __device__ __forceinline__ Cx<R> mul_conj(Cx<R> a, Cx<R> b) {
+    return {a.r * b.r + a.i * b.i, a.i * b.r - a.r * b.i};
+}
+// conj(a) * b
+template <typename R> __device__ __forceinline__ Cx<R> conj_mul(Cx<R> a, Cx<R> b) {
+    return {a.r * b.r + a.i * b.i, a.r * b.i - a.i * b.r};
+}
+// i * a
+template <typename R> __device__ __forceinline__ Cx<R> times_i(Cx<R> a) { return {-a.i, a.r}; }
+template <typename R> __device__ __forceinline__ R norm2(Cx<R> a) { return a.r * a.r + a.i * a.i; }
+
+// ----------------------------------------------------------------------------- precision traits
+template <int P> struct Prec;
+template <> struct Prec<8> { using R = double; };
+template <> struct Prec<4> { using R = float; };
+template <> struct Prec<2> { using R = float; };
+
+constexpr float kHalfMax = 32767.0f;
+constexpr float kHalfInv = 1.0f / 32767.0f;
+
+// cache-policy helpers: streamed data (links, clover) bypasses L1 allocation
+__device__ __forceinline__ float4 ld_stream(const float4 *p) {
+    float4 v;
+    asm volatile("ld.global.nc.L1::no_allocate.v4.f32 {%0,%1,%2,%3}, [%4];"
+                 : "=f"(v.x), "=f"(v.y), "=f"(v.z), "=f"(v.w) : "l"(p));
+    return v;
+}
+__device__ __forceinline__ double2 ld_stream(const double2 *p) {
+    double2 v;
+    asm volatile("ld.global.nc.L1::no_allocate.v2.f64 {%0,%1}, [%2];" : "=d"(v.x), "=d"(v.y) : "l"(p));
+    return v;
+}
+__device__ __forceinline__ float2 ld_stream(const float2 *p) {
+    float2 v;
+    asm volatile("ld.global.nc.L1::no_allocate.v2.f32 {%0,%1}, [%2];" : "=f"(v.x), "=f"(v.y) : "l"(p));
+    return v;
+}
+__device__ __forceinline__ short4 ld_stream(const short4 *p) {
+    short4 v;
+    asm volatile("ld.global.nc.L1::no_allocate.v4.s16 {%0,%1,%2,%3}, [%4];"
+                 : "=h"(v.x), "=h"(v.y), "=h"(v.z), "=h"(v.w) : "l"(p));
+    return v;
+}
+__device__ __forceinline__ short2 ld_stream(const short2 *p) {
+    short2 v;
+    asm volatile("ld.global.nc.L1::no_allocate.v2.s16 {%0,%1}, [%2];" : "=h"(v.x), "=h"(v.y) : "l"(p));
+    return v;
+}
+
+// ----------------------------------------------------------------------------- SoA access
+// Load reals [4*b0, 4*(b0+nb)) (fp32/half) or [2*b0, 2*(b0+nb)) (fp64) of site i.
+// `stream` selects the no-L1-allocate path (links, clover) vs the read-only cached path.
+template <int P, int NB, bool STREAM>
+struct Blocks;
+
+template <int NB, bool STREAM>
+struct Blocks<8, NB, STREAM> {
+    static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, double *out) {
+        const double2 *p = reinterpret_cast<const double2 *>(base);
+#pragma unroll
+        for (int k = 0; k < NB; ++k) {
+            double2 v = STREAM ? ld_stream(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
+            out[2 * k] = v.x;
+            out[2 * k + 1] = v.y;
+        }
+    }
+    static __device__ __forceinline__ void store(void *base, long stride, long i, int b0, const double *in) {
+        double2 *p = reinterpret_cast<double2 *>(base);
+#pragma unroll
+        for (int k = 0; k < NB; ++k) p[(b0 + k) * stride + i] = make_double2(in[2 * k], in[2 * k + 1]);
+    }
+};
+
+template <int NB, bool STREAM>
+struct Blocks<4, NB, STREAM> {
+    static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out) {
+        const float4 *p = reinterpret_cast<const float4 *>(base);
+#pragma unroll
+        for (int k = 0; k < NB; ++k) {
+            float4 v = STREAM ? ld_stream(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
+            out[4 * k] = v.x;
+            out[4 * k + 1] = v.y;
+            out[4 * k + 2] = v.z;
+            out[4 * k + 3] = v.w;
+        }
+    }
+    static __device__ __forceinline__ void store(void *base, long stride, long i, int b0, const float *in) {
+        float4 *p = reinterpret_cast<float4 *>(base);
+#pragma unroll
+        for (int k = 0; k < NB; ++k) p[(b0 + k) * stride + i] = make_float4(in[4 * k], in[4 * k + 1], in[4 * k + 2], in[4 * k + 3]);
+    }
+};
+
+// half: raw integer values scaled by `scale` (norm/32767 for spinors, 1/32767 for links)
+template <int NB, bool STREAM>
+struct Blocks<2, NB, STREAM> {
+    static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out,
+                                                float scale) {
+        const short4 *p = reinterpret_cast<const short4 *>(base);
+#pragma unroll
+        for (int k = 0; k < NB; ++k) {
+            short4 v = STREAM ? ld_stream(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
+            out[4 * k] = scale * (float)v.x;
+            out[4 * k + 1] = scale * (float)v.y;
+            out[4 * k + 2] = scale * (float)v.z;
+            out[4 * k + 3] = scale * (float)v.w;
+        }
+    }
+    static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out) {
+        load(base, stride, i, b0, out, kHalfInv);
+    }
+    // store already-quantised values
+    static __device__ __forceinline__ void store_q(void *base, long stride, long i, int b0, const float *in,
+                                                   float inv_scale) {
+        short4 *p = reinterpret_cast<short4 *>(base);
+#pragma unroll
+        for (int k = 0; k < NB; ++k) {
+            short4 v;
+            v.x = (short)__float2int_rn(in[4 * k] * inv_scale);
+            v.y = (short)__float2int_rn(in[4 * k + 1] * inv_scale);
+            v.z = (short)__float2int_rn(in[4 * k + 2] * inv_scale);
+            v.w = (short)__float2int_rn(in[4 * k + 3] * inv_scale);
+            p[(b0 + k) * stride + i] = v;
+        }
+    }
+};
+
+// ----------------------------------------------------------------------------- spinors
+// A spinor field: 24 reals per site (spin-major, colour, re/im) in the NR basis.
+// fp64: 12 double2 blocks; fp32: 6 float4 blocks; half: 6 short4 blocks + float norm[stride].
+template <int P>
+struct SpinorIO {
+    using R = typename Prec<P>::R;
+    static constexpr int BPH = (P == 8) ? 6 : 3;  // blocks per 12-real half-spinor
+
+    // norm array (half only) follows the 6 short4 blocks
+    static __device__ __forceinline__ const float *norms(const void *base, long stride) {
+        return reinterpret_cast<const float *>(reinterpret_cast<const char *>(base) + (size_t)6 * 8 * stride);
+    }
+    static __device__ __forceinline__ float *norms(void *base, long stride) {
+        return reinterpret_cast<float *>(reinterpret_cast<char *>(base) + (size_t)6 * 8 * stride);
+    }
+
+    // half = 0: reals 0..11 (spins 0,1), half = 1: reals 12..23 (spins 2,3)
+    static __device__ __forceinline__ void load_half(const void *base, long stride, long i, int half, R *out) {
+        if constexpr (P == 2) {
+            float nrm = __ldg(norms(base, stride) + i);
+            Blocks<2, 3, false>::load(base, stride, i, 3 * half, out, nrm * kHalfInv);
+        } else {
+            Blocks<P, BPH, false>::load(base, stride, i, BPH * half, out);
+        }
+    }
+    static __device__ __forceinline__ void load(const void *base, long stride, long i, R *out) {
+        load_half(base, stride, i, 0, out);
+        load_half(base, stride, i, 1, out + 12);
+    }
+    static __device__ __forceinline__ void store(void *base, long stride, long i, const R *in) {
+        if constexpr (P == 2) {
+            float m = 0.f;
+#pragma unroll
+            for (int k = 0; k < 24; ++k) m = fmaxf(m, fabsf(in[k]));
+            norms(base, stride)[i] = m;
+            float inv = (m > 0.f) ? kHalfMax / m : 0.f;
+            Blocks<2, 6, false>::store_q(base, stride, i, 0, in, inv);
+        } else {
+            Blocks<P, 2 * BPH, false>::store(base, stride, i, 0, in);
+        }
+    }
+};
+
+// A face (12 reals per site): fp64 6 double2, fp32 3 float4, half 3 short4 + float norm[fstride]
+template <int P>
+struct FaceIO {
+    using R = typename Prec<P>::R;
+    static constexpr int NB = (P == 8) ? 6 : 3;
+    static __device__ __forceinline__ const float *norms(const void *base, long fs) {
+        return reinterpret_cast<const float *>(reinterpret_cast<const char *>(base) + (size_t)3 * 8 * fs);
+    }
+    static __device__ __forceinline__ float *norms(void *base, long fs) {
+        return reinterpret_cast<float *>(reinterpret_cast<char *>(base) + (size_t)3 * 8 * fs);
+    }
+    static __device__ __forceinline__ void load(const void *base, long fs, long f, R *out) {
+        if constexpr (P == 2) {
+            float nrm = __ldg(norms(base, fs) + f);
+            Blocks<2, 3, false>::load(base, fs, f, 0, out, nrm * kHalfInv);
+        } else {
+            Blocks<P, NB, false>::load(base, fs, f, 0, out);
+        }
+    }
+};
+
+// ----------------------------------------------------------------------------- links
+// Stored reals per link: 18: u[r][c] (re,im); 12: rows 0,1; 8: (theta0, theta2, u01, u02, u10)
+// with theta0 = arg u00, theta2 = arg u20 (half: theta/pi).  Reconstruction in registers:
+// two-row: row2 = conj(row0 x row1); eight-parameter: reading Q6.
+template <int P, int RECON>
+struct LinkIO {
+    using R = typename Prec<P>::R;
+    static __device__ __forceinline__ void load_raw(const void *base, long stride, long i, R *raw) {
+        constexpr int NB4 = (P == 8) ? RECON / 2 : RECON / 4;
+        Blocks<P, NB4, true>::load(base, stride, i, 0, raw);
+        if constexpr (P != 8 && (RECON % 4) != 0) {
+            // trailing 2-real block (recon 18)
+            if constexpr (P == 4) {
+                const float2 *p2 = reinterpret_cast<const float2 *>(reinterpret_cast<const char *>(base) +
+                                                                    (size_t)NB4 * 16 * stride);
+                float2 v = ld_stream(p2 + i);
+                raw[RECON - 2] = v.x;
+                raw[RECON - 1] = v.y;
+            } else {
+                const short2 *p2 = reinterpret_cast<const short2 *>(reinterpret_cast<const char *>(base) +
+                                                                    (size_t)NB4 * 8 * stride);
+                short2 v = ld_stream(p2 + i);
+                raw[RECON - 2] = kHalfInv * (float)v.x;
+                raw[RECON - 1] = kHalfInv * (float)v.y;
+            }
+        }
+    }
+
+    // full 3x3 link u[row][col]
+    static __device__ __forceinline__ void load(const void *base, long stride, long i, Cx<R> u[3][3]) {
+        R raw[RECON];
+        load_raw(base, stride, i, raw);
+        if constexpr (RECON == 18) {
+#pragma unroll
+            for (int r = 0; r < 3; ++r)
+#pragma unroll
+                for (int c = 0; c < 3; ++c) u[r][c] = cx(raw[(r * 3 + c) * 2], raw[(r * 3 + c) * 2 + 1]);
+        } else if constexpr (RECON == 12) {
+#pragma unroll
+            for (int r = 0; r < 2; ++r)
+#pragma unroll
+                for (int c = 0; c < 3; ++c) u[r][c] = cx(raw[(r * 3 + c) * 2], raw[(r * 3 + c) * 2 + 1]);
+            // row2 = conj(row0 x row1)
+            u[2][0] = conj(u[0][1] * u[1][2] - u[0][2] * u[1][1]);
+            u[2][1] = conj(u[0][2] * u[1][0] - u[0][0] * u[1][2]);
+            u[2][2] = conj(u[0][0] * u[1][1] - u[0][1] * u[1][0]);
+        } else {
+            R th0 = raw[0], th2 = raw[1];
+            if constexpr (P == 2) {
+                th0 *= (R)3.14159265358979323846;
+                th2 *= (R)3.14159265358979323846;
+            }
+            Cx<R> u01 = cx(raw[2], raw[3]), u02 = cx(raw[4], raw[5]), u10 = cx(raw[6], raw[7]);
+            R n = norm2(u01) + norm2(u02);
+            R a00 = sqrt(fmax((R)0, (R)1 - n));
+            R s0, c0, s2, c2;
+            sincos_(th0, &s0, &c0);
+            sincos_(th2, &s2, &c2);
+            Cx<R> u00 = cx(a00 * c0, a00 * s0);
+            R a20 = sqrt(fmax((R)0, (R)1 - a00 * a00 - norm2(u10)));
+            Cx<R> u20 = cx(a20 * c2, a20 * s2);
+            R inv = (R)1 / n;
+            Cx<R> A = conj_mul(u00, u10);
+            Cx<R> C = conj_mul(u00, u20);
+            Cx<R> cu20 = conj(u20), cu10 = conj(u10), cu01 = conj(u01), cu02 = conj(u02);
+            u[0][0] = u00; u[0][1] = u01; u[0][2] = u02;
+            u[1][0] = u10;
+            u[2][0] = u20;
+            u[1][1] = (-inv) * (cu20 * cu02 + A * u01);
+            u[1][2] = inv * (cu20 * cu01 - A * u02);
+            u[2][1] = inv * (cu10 * cu02 - C * u01);
+            u[2][2] = (-inv) * (cu10 * cu01 + C * u02);
+        }
+    }
+
+    static __device__ __forceinline__ void sincos_(double x, double *s, double *c) { sincos(x, s, c); }
+    static __device__ __forceinline__ void sincos_(float x, float *s, float *c) { sincosf(x, s, c); }
+};
+
+}  // namespace qx

@@ -1,0 +1,356 @@
+// dslash.cuh — the Wilson-clover Dslash stencil (eq. (2); kernel structure
+// P:384-395), one thread per output site of parity p.
+//
+// Per site x of parity p, for each of the 8 hops: load the link (reconstructing 12/8-real
+// storage in registers), load the neighbour spinor of parity 1-p (24 reals for
+// x, y, z; only the 12 reals selected by the diagonal temporal projector for t, eq. (6),
+// P:504-506), spin-project to a half spinor (footnote 3), multiply by U or U^dag
+// (the backward link U_mu(x-mu) is read at x-mu and conjugated by register relabeling,
+// P:425-432), expand and accumulate.  The clover term is fused before the store.
+//
+// Spin basis: non-relativistic, psi_NR = S psi_DR with S = (1/sqrt2)[[1,1],[1,-1]] (2x2
+// blocks of spin pairs), so 1 + gamma_4 = diag(2,2,0,0) and 1 - gamma_4 = diag(0,0,2,2).
+// Projectors (1 + sigma gamma_mu), sigma = +-1, written as h = (h0, h1) and the
+// reconstruction of rows 2, 3 (derived from gamma_mu^NR = S gamma_mu^DR S):
+//   mu=x: h0 = p0 - s i p3, h1 = p1 - s i p2;   r2 =  s i h1, r3 =  s i h0
+//   mu=y: h0 = p0 + s p3,   h1 = p1 - s p2;     r2 = -s h1,   r3 =  s h0
+//   mu=z: h0 = p0 - s i p2, h1 = p1 + s i p3;   r2 =  s i h0, r3 = -s i h1
+// Non-dagger: forward hop uses 1 - gamma (s = -1), backward 1 + gamma (s = +1) (eq. (2));
+// the dagger flips s (D^dag = gamma5 D gamma5).
+//
+// Clover (72 reals = two Hermitian 6x6 chiral blocks C+, C-, each d[6] + lower triangle
+// L[15]; stored already halved): with u = spins 0,1 and l = spins 2,3 of the NR spinor,
+//   out_u = C+ (u + l) + C- (u - l),  out_l = C+ (u + l) - C- (u - l).
+#pragma once
+#include "core.cuh"
+#include "internal.h"
+
+namespace qx {
+
+template <typename R>
+__device__ __forceinline__ void su3_mul(const Cx<R> u[3][3], const Cx<R> v[3], Cx<R> out[3]) {
+#pragma unroll
+    for (int a = 0; a < 3; ++a) out[a] = u[a][0] * v[0] + u[a][1] * v[1] + u[a][2] * v[2];
+}
+template <typename R>
+__device__ __forceinline__ void su3_dag_mul(const Cx<R> u[3][3], const Cx<R> v[3], Cx<R> out[3]) {
+#pragma unroll
+    for (int a = 0; a < 3; ++a) out[a] = conj_mul(u[0][a], v[0]) + conj_mul(u[1][a], v[1]) + conj_mul(u[2][a], v[2]);
+}
+
+template <typename R>
+__device__ __forceinline__ void unpack_spinor(const R *v, Cx<R> p[4][3]) {
+#pragma unroll
+    for (int s = 0; s < 4; ++s)
+#pragma unroll
+        for (int c = 0; c < 3; ++c) p[s][c] = cx(v[(s * 3 + c) * 2], v[(s * 3 + c) * 2 + 1]);
+}
+
+// spatial hop: project psi with (1 + sigma gamma_mu), multiply by U (or U^dag), accumulate
+template <int MU, int SIGMA, bool ADJ, typename R>
+__device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3][3], R coef, Cx<R> acc[4][3]) {
+    Cx<R> h0[3], h1[3];
+#pragma unroll
+    for (int c = 0; c < 3; ++c) {
+        if constexpr (MU == 0) {
+            Cx<R> a = times_i(p[3][c]), b = times_i(p[2][c]);
+            h0[c] = SIGMA > 0 ? p[0][c] - a : p[0][c] + a;
+            h1[c] = SIGMA > 0 ? p[1][c] - b : p[1][c] + b;
+        } else if constexpr (MU == 1) {
+            h0[c] = SIGMA > 0 ? p[0][c] + p[3][c] : p[0][c] - p[3][c];
+            h1[c] = SIGMA > 0 ? p[1][c] - p[2][c] : p[1][c] + p[2][c];
+        } else {
+            Cx<R> a = times_i(p[2][c]), b = times_i(p[3][c]);
+            h0[c] = SIGMA > 0 ? p[0][c] - a : p[0][c] + a;
+            h1[c] = SIGMA > 0 ? p[1][c] + b : p[1][c] - b;
+        }
+    }
+    Cx<R> g0[3], g1[3];
+    if constexpr (ADJ) {
+        su3_dag_mul(u, h0, g0);
+        su3_dag_mul(u, h1, g1);
+    } else {
+        su3_mul(u, h0, g0);
+        su3_mul(u, h1, g1);
+    }
+#pragma unroll
+    for (int c = 0; c < 3; ++c) {
+        g0[c] = coef * g0[c];
+        g1[c] = coef * g1[c];
+        acc[0][c] = acc[0][c] + g0[c];
+        acc[1][c] = acc[1][c] + g1[c];
+        if constexpr (MU == 0) {
+            Cx<R> a = times_i(g1[c]), b = times_i(g0[c]);
+            acc[2][c] = SIGMA > 0 ? acc[2][c] + a : acc[2][c] - a;
+            acc[3][c] = SIGMA > 0 ? acc[3][c] + b : acc[3][c] - b;
+        } else if constexpr (MU == 1) {
+            acc[2][c] = SIGMA > 0 ? acc[2][c] - g1[c] : acc[2][c] + g1[c];
+            acc[3][c] = SIGMA > 0 ? acc[3][c] + g0[c] : acc[3][c] - g0[c];
+        } else {
+            Cx<R> a = times_i(g0[c]), b = times_i(g1[c]);
+            acc[2][c] = SIGMA > 0 ? acc[2][c] + a : acc[2][c] - a;
+            acc[3][c] = SIGMA > 0 ? acc[3][c] - b : acc[3][c] + b;
+        }
+    }
+}
+
+// temporal hop: h = the 12 selected reals (upper half if UPPER); result 2 U h into the same half
+template <bool UPPER, bool ADJ, typename R>
+__device__ __forceinline__ void temporal_hop(const R *hv, const Cx<R> u[3][3], R coef, Cx<R> acc[4][3]) {
+    Cx<R> h0[3], h1[3], g0[3], g1[3];
+#pragma unroll
+    for (int c = 0; c < 3; ++c) {
+        h0[c] = cx(hv[c * 2], hv[c * 2 + 1]);
+        h1[c] = cx(hv[6 + c * 2], hv[6 + c * 2 + 1]);
+    }
+    if constexpr (ADJ) {
+        su3_dag_mul(u, h0, g0);
+        su3_dag_mul(u, h1, g1);
+    } else {
+        su3_mul(u, h0, g0);
+        su3_mul(u, h1, g1);
+    }
+    constexpr int s0 = UPPER ? 0 : 2;
+#pragma unroll
+    for (int c = 0; c < 3; ++c) {
+        acc[s0][c] = acc[s0][c] + coef * g0[c];
+        acc[s0 + 1][c] = acc[s0 + 1][c] + coef * g1[c];
+    }
+}
+
+// Hermitian 6x6 (d[6], lower triangle L[15]) times v
+template <typename R>
+__device__ __forceinline__ void herm6_mul(const R *m, const Cx<R> v[6], Cx<R> out[6]) {
+#pragma unroll
+    for (int i = 0; i < 6; ++i) out[i] = m[i] * v[i];
+#pragma unroll
+    for (int i = 1; i < 6; ++i)
+#pragma unroll
+        for (int j = 0; j < i; ++j) {
+            const int k = i * (i - 1) / 2 + j;
+            Cx<R> L = cx(m[6 + 2 * k], m[6 + 2 * k + 1]);
+            out[i] = out[i] + L * v[j];
+            out[j] = out[j] + conj_mul(L, v[i]);
+        }
+}
+
+template <int P>
+struct CloverIO {
+    using R = typename Prec<P>::R;
+    // chiral block b (0: C+, 1: C-) of site i: 36 reals
+    static __device__ __forceinline__ void load(const void *base, long stride, long i, int b, R *m) {
+        if constexpr (P == 8) {
+            Blocks<8, 18, true>::load(base, stride, i, 18 * b, m);
+        } else if constexpr (P == 4) {
+            Blocks<4, 9, true>::load(base, stride, i, 9 * b, m);
+        } else {
+            const float2 *nrm = reinterpret_cast<const float2 *>(reinterpret_cast<const char *>(base) +
+                                                                 (size_t)18 * 8 * stride);
+            float2 n = ld_stream(nrm + i);
+            Blocks<2, 9, true>::load(base, stride, i, 9 * b, m, (b ? n.y : n.x) * kHalfInv);
+        }
+    }
+};
+
+template <int P>
+__device__ __forceinline__ void apply_clover(const void *cl, long stride, long i, const Cx<typename Prec<P>::R> in[4][3],
+                                             Cx<typename Prec<P>::R> out[4][3]) {
+    using R = typename Prec<P>::R;
+    Cx<R> va[6], vb[6], wa[6], wb[6];
+#pragma unroll
+    for (int s = 0; s < 2; ++s)
+#pragma unroll
+        for (int c = 0; c < 3; ++c) {
+            va[s * 3 + c] = in[s][c] + in[s + 2][c];
+            vb[s * 3 + c] = in[s][c] - in[s + 2][c];
+        }
+    {
+        R m[36];
+        CloverIO<P>::load(cl, stride, i, 0, m);
+        herm6_mul(m, va, wa);
+    }
+    {
+        R m[36];
+        CloverIO<P>::load(cl, stride, i, 1, m);
+        herm6_mul(m, vb, wb);
+    }
+#pragma unroll
+    for (int s = 0; s < 2; ++s)
+#pragma unroll
+        for (int c = 0; c < 3; ++c) {
+            out[s][c] = wa[s * 3 + c] + wb[s * 3 + c];
+            out[s + 2][c] = wa[s * 3 + c] - wb[s * 3 + c];
+        }
+}
+
+template <int P, int RECON, bool DAG, int KIND>
+__global__ void __launch_bounds__(128) dslash_kernel(const __grid_constant__ DslashArgs a) {
+    using R = typename Prec<P>::R;
+    const int tid = blockIdx.x * blockDim.x + threadIdx.x;
+    if (tid >= a.nthreads) return;
+    int i;
+    if (a.range == RANGE_ALL) i = tid;
+    else if (a.range == RANGE_INTERIOR) i = a.F + tid;
+    else i = (tid < a.F) ? tid : (a.T_loc - 1) * a.F + (tid - a.F);
+
+    const int X = a.X, Y = a.Y, Z = a.Z, Xh = a.Xh;
+    int xh = i % Xh;
+    int r = i / Xh;
+    const int y = r % Y;
+    r /= Y;
+    const int z = r % Z;
+    const int t = r / Z;
+    const int x = 2 * xh + ((a.parity + y + z + t) & 1);
+    const int p = a.parity, op = 1 - p;
+    const int XY = X * Y;
+    const int XYZ = XY * Z;
+    const int lex = ((t * Z + z) * Y + y) * X + x;
+
+    Cx<R> acc[4][3];
+#pragma unroll
+    for (int s = 0; s < 4; ++s)
+#pragma unroll
+        for (int c = 0; c < 3; ++c) acc[s][c] = cx((R)0, (R)0);
+
+    constexpr int SF = DAG ? +1 : -1;  // sigma of the forward hop
+    constexpr int SB = -SF;
+
+    // ---- x direction
+    {
+        const int nf = (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1;
+        const int nb = (x == 0 ? lex + (X - 1) : lex - 1) >> 1;
+        R v[24];
+        Cx<R> ps[4][3], u[3][3];
+        SpinorIO<P>::load(a.in, a.stride, nf, v);
+        unpack_spinor(v, ps);
+        LinkIO<P, RECON>::load(a.gauge[0][p], a.stride, i, u);
+        spatial_hop<0, SF, false>(ps, u, (R)1, acc);
+        SpinorIO<P>::load(a.in, a.stride, nb, v);
+        unpack_spinor(v, ps);
+        LinkIO<P, RECON>::load(a.gauge[0][op], a.stride, nb, u);
+        spatial_hop<0, SB, true>(ps, u, (R)1, acc);
+    }
+    // ---- y direction
+    {
+        const int nf = (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1;
+        const int nb = (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1;
+        R v[24];
+        Cx<R> ps[4][3], u[3][3];
+        SpinorIO<P>::load(a.in, a.stride, nf, v);
+        unpack_spinor(v, ps);
+        LinkIO<P, RECON>::load(a.gauge[1][p], a.stride, i, u);
+        spatial_hop<1, SF, false>(ps, u, (R)1, acc);
+        SpinorIO<P>::load(a.in, a.stride, nb, v);
+        unpack_spinor(v, ps);
+        LinkIO<P, RECON>::load(a.gauge[1][op], a.stride, nb, u);
+        spatial_hop<1, SB, true>(ps, u, (R)1, acc);
+    }
+    // ---- z direction
+    {
+        const int nf = (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1;
+        const int nb = (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1;
+        R v[24];
+        Cx<R> ps[4][3], u[3][3];
+        SpinorIO<P>::load(a.in, a.stride, nf, v);
+        unpack_spinor(v, ps);
+        LinkIO<P, RECON>::load(a.gauge[2][p], a.stride, i, u);
+        spatial_hop<2, SF, false>(ps, u, (R)1, acc);
+        SpinorIO<P>::load(a.in, a.stride, nb, v);
+        unpack_spinor(v, ps);
+        LinkIO<P, RECON>::load(a.gauge[2][op], a.stride, nb, u);
+        spatial_hop<2, SB, true>(ps, u, (R)1, acc);
+    }
+    // ---- t direction: diagonal projectors, 12 reals per neighbour (eq. (6))
+    {
+        // forward: (1 + SF gamma_4): SF = -1 -> lower spins, SF = +1 -> upper spins
+        constexpr bool FWD_UPPER = (SF > 0);
+        const int T_loc = a.T_loc;
+        R h[12];
+        Cx<R> u[3][3];
+        R cf = (R)2;
+        if (t == T_loc - 1) {
+            cf = (R)(2.0 * a.bc_fwd);
+            if (a.ghosted) {
+                FaceIO<P>::load(a.ghost_fwd, a.fstride, i - t * a.F, h);
+            } else {
+                SpinorIO<P>::load_half(a.in, a.stride, (lex - (T_loc - 1) * XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
+            }
+        } else {
+            SpinorIO<P>::load_half(a.in, a.stride, (lex + XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
+        }
+        LinkIO<P, RECON>::load(a.gauge[3][p], a.stride, i, u);
+        temporal_hop<FWD_UPPER, false>(h, u, cf, acc);
+
+        // backward: (1 + SB gamma_4)
+        constexpr bool BWD_UPPER = (SB > 0);
+        R cb = (R)2;
+        if (t == 0) {
+            cb = (R)(2.0 * a.bc_back);
+            if (a.ghosted) {
+                FaceIO<P>::load(a.ghost_back, a.fstride, i, h);
+                LinkIO<P, RECON>::load(a.gauge_ghost, a.fstride, i, u);
+            } else {
+                const int nb = (lex + (T_loc - 1) * XYZ) >> 1;
+                SpinorIO<P>::load_half(a.in, a.stride, nb, BWD_UPPER ? 0 : 1, h);
+                LinkIO<P, RECON>::load(a.gauge[3][op], a.stride, nb, u);
+            }
+        } else {
+            const int nb = (lex - XYZ) >> 1;
+            SpinorIO<P>::load_half(a.in, a.stride, nb, BWD_UPPER ? 0 : 1, h);
+            LinkIO<P, RECON>::load(a.gauge[3][op], a.stride, nb, u);
+        }
+        temporal_hop<BWD_UPPER, true>(h, u, cb, acc);
+    }
+
+    // ---- epilogue: fused clover
+    Cx<R> res[4][3];
+    if constexpr (KIND == QUDAX_HOP) {
+#pragma unroll
+        for (int s = 0; s < 4; ++s)
+#pragma unroll
+            for (int c = 0; c < 3; ++c) res[s][c] = acc[s][c];
+    } else if constexpr (KIND == QUDAX_CLOVER_INV) {
+        apply_clover<P>(a.clover, a.stride, i, acc, res);
+    } else {
+        R v[24];
+        Cx<R> xs[4][3];
+        SpinorIO<P>::load(a.x, a.stride, i, v);
+        unpack_spinor(v, xs);
+        apply_clover<P>(a.clover, a.stride, i, xs, res);
+        const R co = (R)a.a;
+#pragma unroll
+        for (int s = 0; s < 4; ++s)
+#pragma unroll
+            for (int c = 0; c < 3; ++c) res[s][c] = res[s][c] + co * acc[s][c];
+    }
+    R o[24];
+#pragma unroll
+    for (int s = 0; s < 4; ++s)
+#pragma unroll
+        for (int c = 0; c < 3; ++c) {
+            o[(s * 3 + c) * 2] = res[s][c].r;
+            o[(s * 3 + c) * 2 + 1] = res[s][c].i;
+        }
+    SpinorIO<P>::store(a.out, a.stride, i, o);
+}
+
+template <int P>
+void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
+    const int threads = 128;
+    const int blocks = (a.nthreads + threads - 1) / threads;
+    if (blocks == 0) return;
+#define QX_DS(RC, DG, KD)                                                     \
+    if (recon == RC && dagger == DG && kind == KD) {                          \
+        dslash_kernel<P, RC, DG, KD><<<blocks, threads, 0, s>>>(a);           \
+        return;                                                               \
+    }
+#define QX_DS_K(RC, DG) QX_DS(RC, DG, 0) QX_DS(RC, DG, 1) QX_DS(RC, DG, 2)
+#define QX_DS_D(RC) QX_DS_K(RC, false) QX_DS_K(RC, true)
+    QX_DS_D(18) QX_DS_D(12) QX_DS_D(8)
+#undef QX_DS_D
+#undef QX_DS_K
+#undef QX_DS
+    throw Error(QUDAX_ERR_ARG, "dslash: unsupported recon/kind");
+}
+
+}  // namespace qx

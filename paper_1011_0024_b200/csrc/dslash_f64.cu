@@ -1,0 +1,9 @@
+// dslash_f64.cu — instantiation of the Dslash kernel family for storage precision 8 bytes/real
+// (split per precision so the 18 variants per precision compile in parallel).
+#include "dslash.cuh"
+
+namespace qx {
+void launch_dslash_f64(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
+    launch_dslash_prec<8>(recon, dagger, kind, a, s);
+}
+}  // namespace qx

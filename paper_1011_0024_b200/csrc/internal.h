@@ -1,0 +1,129 @@
+// internal.h — host-side declarations shared by the C++ runtime and the CUDA kernels.
+// Not part of the ABI (see include/qudax.h).
+#pragma once
+
+#include <cuda_runtime.h>
+
+#include <cstddef>
+#include <cstdint>
+#include <stdexcept>
+#include <string>
+
+#include "qudax.h"
+
+namespace qx {
+
+// ----------------------------------------------------------------------------- errors
+struct Error : std::runtime_error {
+    qudax_status status;
+    Error(qudax_status s, const std::string &m) : std::runtime_error(m), status(s) {}
+};
+
+#define QX_CUDA(call)                                                                        \
+    do {                                                                                     \
+        cudaError_t e_ = (call);                                                             \
+        if (e_ != cudaSuccess)                                                               \
+            throw ::qx::Error(e_ == cudaErrorMemoryAllocation ? QUDAX_ERR_OOM : QUDAX_ERR_CUDA, \
+                              std::string(#call) + ": " + cudaGetErrorString(e_));          \
+    } while (0)
+
+#define QX_CHECK(cond, status, msg)                          \
+    do {                                                     \
+        if (!(cond)) throw ::qx::Error((status), (msg));     \
+    } while (0)
+
+// ----------------------------------------------------------------------------- layouts
+// Site-major SoA (eq. (4)): a field with N reals per site is stored as blocks of
+// 16-byte (fp64, fp32) or 8-byte (half) vectors; block b, site i lives at
+// base + (b * stride + i) * vec_bytes.  stride = number of sites padded to 64.
+inline long pad64(long n) { return (n + 63) / 64 * 64; }
+
+// bytes of one "N-real" site-major array with `stride` sites in precision prec.
+// fp64: N/2 double2; fp32: N/4 float4 (+1 float2 if N%4==2); half: N/4 short4 (+1 short2).
+inline size_t soa_bytes(int prec, int nreal, long stride) {
+    if (prec == 8) return (size_t)(nreal / 2) * 16 * stride;
+    if (prec == 4) return ((size_t)(nreal / 4) * 16 + (nreal % 4 ? 8 : 0)) * stride;
+    return ((size_t)(nreal / 4) * 8 + (nreal % 4 ? 4 : 0)) * stride;
+}
+// spinor (24 reals) + half norm (one float per site)
+inline size_t spinor_bytes(int prec, long stride) {
+    return soa_bytes(prec, 24, stride) + (prec == 2 ? (size_t)4 * stride : 0);
+}
+// projected face (12 reals) + half norm
+inline size_t face_bytes(int prec, long fstride) {
+    return soa_bytes(prec, 12, fstride) + (prec == 2 ? (size_t)4 * fstride : 0);
+}
+// clover: 72 reals = two 6x6 Hermitian chiral blocks; half adds 2 floats (one per block)
+inline size_t clover_bytes(int prec, long stride) {
+    return soa_bytes(prec, 72, stride) + (prec == 2 ? (size_t)8 * stride : 0);
+}
+
+// ----------------------------------------------------------------------------- geometry
+struct Geom {
+    int X, Y, Z, T;        // global
+    int T_loc, t0, rank, nranks;
+    int Xh;                // X/2
+    long Vs, V, Vh, F;     // X*Y*Z, local volume, V/2, face sites = Vs/2
+    long stride, fstride;  // padded Vh, padded F
+};
+
+// ----------------------------------------------------------------------------- kernels
+enum SiteRange { RANGE_ALL = 0, RANGE_INTERIOR = 1, RANGE_BOUNDARY = 2 };
+
+struct DslashArgs {
+    // geometry
+    int X, Y, Z, T_loc, Xh;
+    int Vh, F;
+    long stride, fstride;
+    int parity;            // output parity p
+    int range;             // SiteRange
+    int ghosted;           // 1: t-hops off the slab read ghost buffers; 0: periodic wrap
+    int nthreads;          // sites this launch covers
+    double bc_fwd, bc_back; // sign on the t-hop out of local t=T_loc-1 (fwd) / t=0 (back)
+    double a;              // xpay coefficient
+    const void *in;        // parity 1-p spinor
+    void *out;             // parity p spinor
+    const void *x;         // parity p spinor (xpay)
+    const void *gauge[4][2];
+    const void *gauge_ghost; // U_t at global t0-1, parity 1-p, face layout (F sites)
+    const void *clover;    // parity p: T (xpay) or T^{-1} (clover_inv)
+    const void *ghost_back; // upper (non-dagger) half-spinors from rank-1, face layout
+    const void *ghost_fwd;  // lower (non-dagger) half-spinors from rank+1
+};
+
+void launch_dslash_f64(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
+void launch_dslash_f32(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
+void launch_dslash_f16(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
+
+// face pack: t_loc = 0 slice half (lower if !dagger) -> send_back; t_loc = T_loc-1 half
+// (upper if !dagger) -> send_fwd.  `in` is the Dslash input field (parity 1-p).
+void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back,
+                       void *send_fwd, cudaStream_t s);
+
+// layout conversion (DR AoS fp64 <-> NR SoA prec), one parity
+void launch_spinor_import(int prec, const Geom &g, int parity, const double *src, void *dst, cudaStream_t s);
+void launch_spinor_export(int prec, const Geom &g, int parity, const void *src, double *dst, cudaStream_t s);
+void launch_spinor_convert(int dst_prec, int src_prec, const Geom &g, void *dst, const void *src, cudaStream_t s);
+
+// gauge: extended fp64 AoS [T_loc+2][4][Z][Y][X][3][3] complex (slot 0 = global t0-1,
+// slot T_loc+1 = t0+T_loc) -> per-mu, per-parity SoA (prec, recon) plus the ghost U_t(t0-1)
+// per site parity (face layout).  *bad counts links with |u01|^2+|u02|^2 < 1e-6 (recon 8).
+void launch_gauge_pack2(int prec, int recon, const Geom &g, const double *ext, void *const dst[4][2],
+                        void *const ghost[2], int *bad, cudaStream_t s);
+// clover: from the extended fp64 gauge, T = 1 + 2 kappa A and T^{-1} as two 6x6 Hermitian
+// chiral blocks per site (fp64 [Vh][72], halved for the NR rotation), both parities.
+void launch_clover_build(const Geom &g, const double *ext, double kappa, double csw, double *T[2],
+                         double *Tinv[2], int *bad_sites, cudaStream_t s);
+void launch_clover_pack(int prec, const Geom &g, const double *src, void *dst, cudaStream_t s);
+void launch_clover_apply(int prec, const Geom &g, const void *cl, const void *in, void *out, cudaStream_t s);
+
+// BLAS / reductions (blas.cu).  ops: 0 p_update, 1 caxpy, 2 xpay, 3 cdot, 4 norm2, 5 tdot,
+// 6 bicgstab final update, 7 r = b - r with |r|^2.  Returns the number of reduced doubles
+// written to `out` (device).
+enum BlasOp { OP_P_UPDATE = 0, OP_CAXPY, OP_XPAY, OP_CDOT, OP_NORM2, OP_TDOT, OP_FINAL, OP_BMR_NORM };
+int blas_run(int op, int prec, const Geom &g, void *const *f, const double *coef, double *partials, double *out,
+             cudaStream_t s);
+void blas_xpy_mixed(int pd, int ps, const Geom &g, const void *x, void *y, cudaStream_t s);
+int blas_partial_blocks();
+
+}  // namespace qx

@@ -1,0 +1,509 @@
+// layout.cu — field reordering and setup kernels (all on the device):
+//  * spinor import/export: host-order DeGrand-Rossi AoS fp64 <-> non-relativistic-basis
+//    site-major SoA in fp64 / fp32 / half (eqs. (3)-(4); eq. (6) basis change,
+//    P:479-506; half-precision encoding, reading Q7), one parity at a time;
+//  * gauge pack: fp64 links -> per-direction, per-parity SoA with 18/12/8-real storage
+//    (reading Q6), plus the backward temporal ghost link face;
+//  * clover build + invert: four-leaf field strength -> T = 1 + 2 kappa A and T^{-1} as two
+//    Hermitian 6x6 chiral blocks per site, fp64 (reading Q1);
+//  * face pack for the T-direction halo.
+#include "core.cuh"
+#include "dslash.cuh"
+#include "internal.h"
+
+namespace qx {
+
+__host__ __device__ constexpr double kInvSqrt2 = 0.70710678118654752440;
+
+// coordinates of cb site i of parity p (local; t0 is even so local parity = global parity)
+struct Coord {
+    int x, y, z, t, lex;
+};
+__device__ __forceinline__ Coord cb_coord(int i, int p, int X, int Y, int Z) {
+    const int Xh = X / 2;
+    Coord c;
+    int xh = i % Xh;
+    int r = i / Xh;
+    c.y = r % Y;
+    r /= Y;
+    c.z = r % Z;
+    c.t = r / Z;
+    c.x = 2 * xh + ((p + c.y + c.z + c.t) & 1);
+    c.lex = ((c.t * Z + c.z) * Y + c.y) * X + c.x;
+    return c;
+}
+
+// ============================================================================ spinors
+template <int P>
+__global__ void k_spinor_import(int X, int Y, int Z, int Vh, long stride, int parity, const double *__restrict__ src,
+                                void *__restrict__ dst) {
+    using R = typename Prec<P>::R;
+    const int i = blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= Vh) return;
+    Coord c = cb_coord(i, parity, X, Y, Z);
+    const double *s = src + (size_t)c.lex * 24;
+    double d[24];
+#pragma unroll
+    for (int k = 0; k < 24; ++k) d[k] = s[k];
+    // psi_NR = S psi_DR: NR0 = (DR0 + DR2)/sqrt2, NR1 = (DR1 + DR3)/sqrt2,
+    //                    NR2 = (DR0 - DR2)/sqrt2, NR3 = (DR1 - DR3)/sqrt2
+    R o[24];
+#pragma unroll
+    for (int k = 0; k < 12; ++k) {  // k runs over (spin in {0,1}) x colour x re/im
+        const double up = d[k], lo = d[k + 12];
+        o[k] = (R)((up + lo) * kInvSqrt2);
+        o[k + 12] = (R)((up - lo) * kInvSqrt2);
+    }
+    SpinorIO<P>::store(dst, stride, i, o);
+}
+
+template <int P>
+__global__ void k_spinor_export(int X, int Y, int Z, int Vh, long stride, int parity, const void *__restrict__ src,
+                                double *__restrict__ dst) {
+    using R = typename Prec<P>::R;
+    const int i = blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= Vh) return;
+    Coord c = cb_coord(i, parity, X, Y, Z);
+    R v[24];
+    SpinorIO<P>::load(src, stride, i, v);
+    double *d = dst + (size_t)c.lex * 24;
+#pragma unroll
+    for (int k = 0; k < 12; ++k) {
+        const double up = (double)v[k], lo = (double)v[k + 12];
+        d[k] = (up + lo) * kInvSqrt2;
+        d[k + 12] = (up - lo) * kInvSqrt2;
+    }
+}
+
+template <int PD, int PS>
+__global__ void k_spinor_convert(int Vh, long stride, void *__restrict__ dst, const void *__restrict__ src) {
+    const int i = blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= Vh) return;
+    typename Prec<PS>::R v[24];
+    SpinorIO<PS>::load(src, stride, i, v);
+    typename Prec<PD>::R o[24];
+#pragma unroll
+    for (int k = 0; k < 24; ++k) o[k] = (typename Prec<PD>::R)v[k];
+    SpinorIO<PD>::store(dst, stride, i, o);
+}
+
+static inline int nblk(long n, int t) { return (int)((n + t - 1) / t); }
+
+void launch_spinor_import(int prec, const Geom &g, int parity, const double *src, void *dst, cudaStream_t s) {
+    const int T = 128;
+    if (prec == 8) k_spinor_import<8><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
+    else if (prec == 4) k_spinor_import<4><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
+    else k_spinor_import<2><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
+    QX_CUDA(cudaGetLastError());
+}
+void launch_spinor_export(int prec, const Geom &g, int parity, const void *src, double *dst, cudaStream_t s) {
+    const int T = 128;
+    if (prec == 8) k_spinor_export<8><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
+    else if (prec == 4) k_spinor_export<4><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
+    else k_spinor_export<2><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
+    QX_CUDA(cudaGetLastError());
+}
+void launch_spinor_convert(int pd, int ps, const Geom &g, void *dst, const void *src, cudaStream_t s) {
+    const int T = 128;
+    const int b = nblk(g.Vh, T);
+    const int n = (int)g.Vh;
+#define QX_CV(A, B) \
+    if (pd == A && ps == B) { k_spinor_convert<A, B><<<b, T, 0, s>>>(n, g.stride, dst, src); QX_CUDA(cudaGetLastError()); return; }
+    QX_CV(8, 8) QX_CV(8, 4) QX_CV(8, 2) QX_CV(4, 8) QX_CV(4, 4) QX_CV(4, 2) QX_CV(2, 8) QX_CV(2, 4) QX_CV(2, 2)
+#undef QX_CV
+    throw Error(QUDAX_ERR_ARG, "convert: bad precision");
+}
+
+// ============================================================================ gauge
+// ext: fp64 complex [T_loc + 2][4][Z][Y][X][3][3]; slot 0 = global t0-1, slot T_loc+1 = t0+T_loc.
+__device__ __forceinline__ const double *ext_link(const double *ext, long Vs, int t_ext, int mu, long slex) {
+    return ext + (((size_t)t_ext * 4 + mu) * Vs + slex) * 18;
+}
+
+template <int P, int RECON>
+__device__ void encode_store_link(const double *l /*18*/, void *base, long stride, long i, int *bad) {
+    double raw[18];
+    int n = 0;
+    if constexpr (RECON == 18) {
+        for (int k = 0; k < 18; ++k) raw[n++] = l[k];
+    } else if constexpr (RECON == 12) {
+        for (int k = 0; k < 12; ++k) raw[n++] = l[k];
+    } else {
+        double th0 = atan2(l[1], l[0]);     // arg u00
+        double th2 = atan2(l[13], l[12]);   // arg u20
+        if constexpr (P == 2) {
+            th0 /= 3.14159265358979323846;
+            th2 /= 3.14159265358979323846;
+        }
+        raw[n++] = th0;
+        raw[n++] = th2;
+        raw[n++] = l[2]; raw[n++] = l[3];   // u01
+        raw[n++] = l[4]; raw[n++] = l[5];   // u02
+        raw[n++] = l[6]; raw[n++] = l[7];   // u10
+        double nn = l[2] * l[2] + l[3] * l[3] + l[4] * l[4] + l[5] * l[5];
+        if (nn < 1e-6) atomicAdd(bad, 1);
+    }
+    if constexpr (P == 8) {
+        double2 *p = reinterpret_cast<double2 *>(base);
+        for (int k = 0; k < RECON / 2; ++k) p[k * stride + i] = make_double2(raw[2 * k], raw[2 * k + 1]);
+    } else if constexpr (P == 4) {
+        float4 *p = reinterpret_cast<float4 *>(base);
+        constexpr int NB = RECON / 4;
+        for (int k = 0; k < NB; ++k)
+            p[k * stride + i] = make_float4((float)raw[4 * k], (float)raw[4 * k + 1], (float)raw[4 * k + 2], (float)raw[4 * k + 3]);
+        if constexpr (RECON % 4) {
+            float2 *q = reinterpret_cast<float2 *>(reinterpret_cast<char *>(base) + (size_t)NB * 16 * stride);
+            q[i] = make_float2((float)raw[RECON - 2], (float)raw[RECON - 1]);
+        }
+    } else {
+        short4 *p = reinterpret_cast<short4 *>(base);
+        constexpr int NB = RECON / 4;
+        auto q16 = [](double v) { return (short)__double2int_rn(v * 32767.0); };
+        for (int k = 0; k < NB; ++k) {
+            short4 v;
+            v.x = q16(raw[4 * k]); v.y = q16(raw[4 * k + 1]); v.z = q16(raw[4 * k + 2]); v.w = q16(raw[4 * k + 3]);
+            p[k * stride + i] = v;
+        }
+        if constexpr (RECON % 4) {
+            short2 *q = reinterpret_cast<short2 *>(reinterpret_cast<char *>(base) + (size_t)NB * 8 * stride);
+            short2 v;
+            v.x = q16(raw[RECON - 2]); v.y = q16(raw[RECON - 1]);
+            q[i] = v;
+        }
+    }
+}
+
+struct GaugeDst {
+    void *d[4][2];
+    void *ghost[2];
+};
+
+template <int P, int RECON>
+__global__ void k_gauge_pack(int X, int Y, int Z, int T_loc, long Vh, long F, long stride, long fstride,
+                             const double *__restrict__ ext, GaugeDst dst, int *bad) {
+    const long Vs = (long)X * Y * Z;
+    const long n_bulk = 8 * Vh;  // (mu, parity, i)
+    const long n_ghost = 2 * F;  // (parity, f)
+    long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    if (k < n_bulk) {
+        const int mu = (int)(k / (2 * Vh));
+        const int p = (int)((k / Vh) % 2);
+        const int i = (int)(k % Vh);
+        Coord c = cb_coord(i, p, X, Y, Z);
+        const long slex = c.lex - (long)c.t * Vs;
+        encode_store_link<P, RECON>(ext_link(ext, Vs, c.t + 1, mu, slex), dst.d[mu][p], stride, i, bad);
+        return;
+    }
+    k -= n_bulk;
+    if (k < n_ghost) {
+        // U_t at global t0 - 1 (ext slot 0), site parity q; face index f = spatial lex / 2
+        const int q = (int)(k / F);
+        const int f = (int)(k % F);
+        const int Xh = X / 2;
+        int xh = f % Xh;
+        int r = f / Xh;
+        const int y = r % Y;
+        const int z = r / Y;
+        const int x = 2 * xh + ((q + y + z + 1) & 1);  // local t = -1 is odd
+        const long slex = ((long)z * Y + y) * X + x;
+        encode_store_link<P, RECON>(ext_link(ext, Vs, 0, 3, slex), dst.ghost[q], fstride, f, bad);
+    }
+}
+
+void launch_gauge_pack2(int prec, int recon, const Geom &g, const double *ext, void *const dst[4][2],
+                        void *const ghost[2], int *bad, cudaStream_t s) {
+    GaugeDst d;
+    for (int m = 0; m < 4; ++m)
+        for (int p = 0; p < 2; ++p) d.d[m][p] = dst[m][p];
+    d.ghost[0] = ghost[0];
+    d.ghost[1] = ghost[1];
+    const long n = 8 * g.Vh + 2 * g.F;
+    const int T = 128;
+    const int b = nblk(n, T);
+#define QX_GP(PP, RR)                                                                                          \
+    if (prec == PP && recon == RR) {                                                                           \
+        k_gauge_pack<PP, RR><<<b, T, 0, s>>>(g.X, g.Y, g.Z, g.T_loc, g.Vh, g.F, g.stride, g.fstride, ext, d, bad); \
+        QX_CUDA(cudaGetLastError());                                                                           \
+        return;                                                                                                \
+    }
+    QX_GP(8, 18) QX_GP(8, 12) QX_GP(8, 8) QX_GP(4, 18) QX_GP(4, 12) QX_GP(4, 8) QX_GP(2, 18) QX_GP(2, 12) QX_GP(2, 8)
+#undef QX_GP
+    throw Error(QUDAX_ERR_ARG, "gauge pack: bad precision/reconstruct");
+}
+
+// ============================================================================ clover
+// DeGrand-Rossi gamma matrices (gamma_4 reproduces eq. (6) left side),
+// entries (re, im).  Product's own copy, written from the convention, not shared.
+__constant__ double c_gamma[4][4][4][2] = {
+    {{{0, 0}, {0, 0}, {0, 0}, {0, 1}}, {{0, 0}, {0, 0}, {0, 1}, {0, 0}}, {{0, 0}, {0, -1}, {0, 0}, {0, 0}}, {{0, -1}, {0, 0}, {0, 0}, {0, 0}}},
+    {{{0, 0}, {0, 0}, {0, 0}, {-1, 0}}, {{0, 0}, {0, 0}, {1, 0}, {0, 0}}, {{0, 0}, {1, 0}, {0, 0}, {0, 0}}, {{-1, 0}, {0, 0}, {0, 0}, {0, 0}}},
+    {{{0, 0}, {0, 0}, {0, 1}, {0, 0}}, {{0, 0}, {0, 0}, {0, 0}, {0, -1}}, {{0, -1}, {0, 0}, {0, 0}, {0, 0}}, {{0, 0}, {0, 1}, {0, 0}, {0, 0}}},
+    {{{0, 0}, {0, 0}, {1, 0}, {0, 0}}, {{0, 0}, {0, 0}, {0, 0}, {1, 0}}, {{1, 0}, {0, 0}, {0, 0}, {0, 0}}, {{0, 0}, {1, 0}, {0, 0}, {0, 0}}},
+};
+
+using Cd = Cx<double>;
+struct M3 {
+    Cd m[3][3];
+};
+__device__ __forceinline__ M3 load_m3(const double *l) {
+    M3 r;
+    for (int a = 0; a < 3; ++a)
+        for (int b = 0; b < 3; ++b) r.m[a][b] = cx(l[(a * 3 + b) * 2], l[(a * 3 + b) * 2 + 1]);
+    return r;
+}
+__device__ __forceinline__ M3 mul(const M3 &A, const M3 &B) {
+    M3 r;
+    for (int a = 0; a < 3; ++a)
+        for (int b = 0; b < 3; ++b) r.m[a][b] = A.m[a][0] * B.m[0][b] + A.m[a][1] * B.m[1][b] + A.m[a][2] * B.m[2][b];
+    return r;
+}
+__device__ __forceinline__ M3 dagm(const M3 &A) {
+    M3 r;
+    for (int a = 0; a < 3; ++a)
+        for (int b = 0; b < 3; ++b) r.m[a][b] = conj(A.m[b][a]);
+    return r;
+}
+
+// Gauss-Jordan inversion of a 6x6 complex matrix with partial pivoting; returns 0 if singular
+__device__ int invert6(Cd a[6][6], Cd inv[6][6]) {
+    for (int i = 0; i < 6; ++i)
+        for (int j = 0; j < 6; ++j) inv[i][j] = cx(i == j ? 1.0 : 0.0, 0.0);
+    for (int c = 0; c < 6; ++c) {
+        int piv = c;
+        double best = norm2(a[c][c]);
+        for (int r = c + 1; r < 6; ++r)
+            if (norm2(a[r][c]) > best) { best = norm2(a[r][c]); piv = r; }
+        if (best < 1e-300) return 0;
+        if (piv != c)
+            for (int j = 0; j < 6; ++j) {
+                Cd t = a[c][j]; a[c][j] = a[piv][j]; a[piv][j] = t;
+                t = inv[c][j]; inv[c][j] = inv[piv][j]; inv[piv][j] = t;
+            }
+        const double dn = 1.0 / norm2(a[c][c]);
+        const Cd ip = cx(a[c][c].r * dn, -a[c][c].i * dn);
+        for (int j = 0; j < 6; ++j) { a[c][j] = ip * a[c][j]; inv[c][j] = ip * inv[c][j]; }
+        for (int r = 0; r < 6; ++r) {
+            if (r == c) continue;
+            const Cd f = a[r][c];
+            for (int j = 0; j < 6; ++j) { a[r][j] = a[r][j] - f * a[c][j]; inv[r][j] = inv[r][j] - f * inv[c][j]; }
+        }
+    }
+    return 1;
+}
+
+// store Hermitian 6x6 (halved) as d[6], lower-triangle L[15] (re, im)
+__device__ void store_herm6_half(const Cd m[6][6], double *out) {
+    for (int i = 0; i < 6; ++i) out[i] = 0.5 * m[i][i].r;
+    for (int i = 1; i < 6; ++i)
+        for (int j = 0; j < i; ++j) {
+            const int k = i * (i - 1) / 2 + j;
+            // symmetrise against rounding: average of m[i][j] and conj(m[j][i])
+            out[6 + 2 * k] = 0.25 * (m[i][j].r + m[j][i].r);
+            out[6 + 2 * k + 1] = 0.25 * (m[i][j].i - m[j][i].i);
+        }
+}
+
+// one thread per local site (both parities); T[p], Tinv[p]: fp64 [Vh][72]
+__global__ void k_clover_build(int X, int Y, int Z, int T_loc, double kappa, double csw, const double *__restrict__ ext,
+                               double *T0, double *T1, double *I0, double *I1, int *bad) {
+    const long Vs = (long)X * Y * Z;
+    const long V = Vs * T_loc;
+    const long lexl = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    if (lexl >= V) return;
+    int c[4];
+    c[0] = (int)(lexl % X);
+    c[1] = (int)((lexl / X) % Y);
+    c[2] = (int)((lexl / ((long)X * Y)) % Z);
+    c[3] = (int)(lexl / Vs);
+    const int dims[4] = {X, Y, Z, T_loc};
+    const int parity = (c[0] + c[1] + c[2] + c[3]) & 1;
+    const long cb = lexl >> 1;
+    // link U_mu at (site + shifts), t in ext coordinates (t_ext = t + 1), spatial periodic
+    auto L = [&](int mu, int dm, int dmv, int nu, int dn) -> M3 {
+        int s[4] = {c[0], c[1], c[2], c[3]};
+        s[dmv] += dm;
+        s[nu] += dn;
+        for (int d = 0; d < 3; ++d) s[d] = (s[d] + dims[d]) % dims[d];
+        const long slex = ((long)s[2] * Y + s[1]) * X + s[0];
+        return load_m3(ext_link(ext, Vs, s[3] + 1, mu, slex));
+    };
+    // block-diagonal chiral pieces of sum_{mu<nu} gamma_mu gamma_nu (x) F_munu
+    Cd Bup[6][6], Blo[6][6];
+    for (int i = 0; i < 6; ++i)
+        for (int j = 0; j < 6; ++j) { Bup[i][j] = cx(0.0, 0.0); Blo[i][j] = cx(0.0, 0.0); }
+    for (int mu = 0; mu < 4; ++mu)
+        for (int nu = mu + 1; nu < 4; ++nu) {
+            // leaves (counter-clockwise in the mu-nu plane, starting and ending at x)
+            M3 l1 = mul(mul(mul(L(mu, 0, mu, nu, 0), L(nu, 1, mu, nu, 0)), dagm(L(mu, 0, mu, nu, 1))), dagm(L(nu, 0, mu, nu, 0)));
+            M3 l2 = mul(mul(mul(L(nu, 0, mu, nu, 0), dagm(L(mu, -1, mu, nu, 1))), dagm(L(nu, -1, mu, nu, 0))), L(mu, -1, mu, nu, 0));
+            M3 l3 = mul(mul(mul(dagm(L(mu, -1, mu, nu, 0)), dagm(L(nu, -1, mu, nu, -1))), L(mu, -1, mu, nu, -1)), L(nu, 0, mu, nu, -1));
+            M3 l4 = mul(mul(mul(dagm(L(nu, 0, mu, nu, -1)), L(mu, 0, mu, nu, -1)), L(nu, 1, mu, nu, -1)), dagm(L(mu, 0, mu, nu, 0)));
+            Cd F[3][3];
+            for (int a = 0; a < 3; ++a)
+                for (int b = 0; b < 3; ++b) {
+                    Cd q = l1.m[a][b] + l2.m[a][b] + l3.m[a][b] + l4.m[a][b];
+                    Cd qd = conj(l1.m[b][a] + l2.m[b][a] + l3.m[b][a] + l4.m[b][a]);
+                    F[a][b] = 0.125 * (q - qd);
+                }
+            // gamma_mu gamma_nu
+            Cd gg[4][4];
+            for (int r = 0; r < 4; ++r)
+                for (int s = 0; s < 4; ++s) {
+                    Cd v = cx(0.0, 0.0);
+                    for (int k = 0; k < 4; ++k)
+                        v = v + cx(c_gamma[mu][r][k][0], c_gamma[mu][r][k][1]) * cx(c_gamma[nu][k][s][0], c_gamma[nu][k][s][1]);
+                    gg[r][s] = v;
+                }
+            for (int r = 0; r < 2; ++r)
+                for (int s = 0; s < 2; ++s)
+                    for (int a = 0; a < 3; ++a)
+                        for (int b = 0; b < 3; ++b) {
+                            Bup[r * 3 + a][s * 3 + b] = Bup[r * 3 + a][s * 3 + b] + gg[r][s] * F[a][b];
+                            Blo[r * 3 + a][s * 3 + b] = Blo[r * 3 + a][s * 3 + b] + gg[r + 2][s + 2] * F[a][b];
+                        }
+        }
+    // T = 1 + 2 kappa A, A = -(csw/2) sum gamma gamma F  ->  T = 1 - kappa csw sum(...)
+    const double coef = -kappa * csw;
+    for (int i = 0; i < 6; ++i)
+        for (int j = 0; j < 6; ++j) {
+            Bup[i][j] = coef * Bup[i][j];
+            Blo[i][j] = coef * Blo[i][j];
+            if (i == j) {
+                Bup[i][j].r += 1.0;
+                Blo[i][j].r += 1.0;
+            }
+        }
+    double *To = parity ? T1 : T0;
+    double *Io = parity ? I1 : I0;
+    store_herm6_half(Bup, To + cb * 72);
+    store_herm6_half(Blo, To + cb * 72 + 36);
+    Cd inv[6][6];
+    if (!invert6(Bup, inv)) atomicAdd(bad, 1);
+    store_herm6_half(inv, Io + cb * 72);
+    if (!invert6(Blo, inv)) atomicAdd(bad, 1);
+    store_herm6_half(inv, Io + cb * 72 + 36);
+}
+
+void launch_clover_build(const Geom &g, const double *ext, double kappa, double csw, double *T[2], double *Tinv[2],
+                         int *bad, cudaStream_t s) {
+    const int TB = 64;
+    k_clover_build<<<nblk(g.V, TB), TB, 0, s>>>(g.X, g.Y, g.Z, g.T_loc, kappa, csw, ext, T[0], T[1], Tinv[0], Tinv[1], bad);
+    QX_CUDA(cudaGetLastError());
+}
+
+// fp64 AoS [Vh][72] -> SoA in prec (half: per-chiral-block float norms)
+template <int P>
+__global__ void k_clover_pack(long Vh, long stride, const double *__restrict__ src, void *__restrict__ dst) {
+    const long i = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= Vh) return;
+    const double *s = src + i * 72;
+    if constexpr (P == 8) {
+        double2 *p = reinterpret_cast<double2 *>(dst);
+        for (int k = 0; k < 36; ++k) p[k * stride + i] = make_double2(s[2 * k], s[2 * k + 1]);
+    } else if constexpr (P == 4) {
+        float4 *p = reinterpret_cast<float4 *>(dst);
+        for (int k = 0; k < 18; ++k)
+            p[k * stride + i] = make_float4((float)s[4 * k], (float)s[4 * k + 1], (float)s[4 * k + 2], (float)s[4 * k + 3]);
+    } else {
+        short4 *p = reinterpret_cast<short4 *>(dst);
+        float2 *nrm = reinterpret_cast<float2 *>(reinterpret_cast<char *>(dst) + (size_t)18 * 8 * stride);
+        float n[2];
+        for (int b = 0; b < 2; ++b) {
+            double m = 0;
+            for (int k = 0; k < 36; ++k) m = fmax(m, fabs(s[36 * b + k]));
+            n[b] = (float)m;
+            const float inv = m > 0 ? kHalfMax / (float)m : 0.f;
+            for (int k = 0; k < 9; ++k) {
+                short4 v;
+                v.x = (short)__float2int_rn((float)s[36 * b + 4 * k] * inv);
+                v.y = (short)__float2int_rn((float)s[36 * b + 4 * k + 1] * inv);
+                v.z = (short)__float2int_rn((float)s[36 * b + 4 * k + 2] * inv);
+                v.w = (short)__float2int_rn((float)s[36 * b + 4 * k + 3] * inv);
+                p[(9 * b + k) * stride + i] = v;
+            }
+        }
+        nrm[i] = make_float2(n[0], n[1]);
+    }
+}
+
+void launch_clover_pack(int prec, const Geom &g, const double *src, void *dst, cudaStream_t s) {
+    const int T = 128;
+    if (prec == 8) k_clover_pack<8><<<nblk(g.Vh, T), T, 0, s>>>(g.Vh, g.stride, src, dst);
+    else if (prec == 4) k_clover_pack<4><<<nblk(g.Vh, T), T, 0, s>>>(g.Vh, g.stride, src, dst);
+    else k_clover_pack<2><<<nblk(g.Vh, T), T, 0, s>>>(g.Vh, g.stride, src, dst);
+    QX_CUDA(cudaGetLastError());
+}
+
+// site-local clover multiply out = C in (C = T or T^{-1} of the field's parity)
+template <int P>
+__global__ void k_clover_apply(long Vh, long stride, const void *__restrict__ cl, const void *__restrict__ in,
+                               void *__restrict__ out) {
+    using R = typename Prec<P>::R;
+    const long i = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= Vh) return;
+    R v[24];
+    SpinorIO<P>::load(in, stride, i, v);
+    Cx<R> ps[4][3], o[4][3];
+    unpack_spinor(v, ps);
+    apply_clover<P>(cl, stride, i, ps, o);
+    for (int s = 0; s < 4; ++s)
+        for (int c = 0; c < 3; ++c) {
+            v[(s * 3 + c) * 2] = o[s][c].r;
+            v[(s * 3 + c) * 2 + 1] = o[s][c].i;
+        }
+    SpinorIO<P>::store(out, stride, i, v);
+}
+
+void launch_clover_apply(int prec, const Geom &g, const void *cl, const void *in, void *out, cudaStream_t s) {
+    const int T = 128;
+    if (prec == 8) k_clover_apply<8><<<nblk(g.Vh, T), T, 0, s>>>(g.Vh, g.stride, cl, in, out);
+    else if (prec == 4) k_clover_apply<4><<<nblk(g.Vh, T), T, 0, s>>>(g.Vh, g.stride, cl, in, out);
+    else k_clover_apply<2><<<nblk(g.Vh, T), T, 0, s>>>(g.Vh, g.stride, cl, in, out);
+    QX_CUDA(cudaGetLastError());
+}
+
+// ============================================================================ faces
+// Raw copy of one 12-real half (3 float4 / 6 double2 / 3 short4 + the site norm): bits only,
+// so a partitioned Dslash reads exactly what the unpartitioned one reads.
+template <int P>
+__global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
+                             const void *__restrict__ in, void *__restrict__ sb, void *__restrict__ sf) {
+    long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    if (k >= 2 * F) return;
+    const bool fwd = k >= F;
+    const long f = fwd ? k - F : k;
+    const long i = fwd ? (T_loc - 1) * F + f : f;
+    void *dst = fwd ? sf : sb;
+    const int half = fwd ? half_fwd : half_back;
+    if constexpr (P == 8) {
+        const double2 *s = reinterpret_cast<const double2 *>(in);
+        double2 *d = reinterpret_cast<double2 *>(dst);
+        for (int b = 0; b < 6; ++b) d[b * fstride + f] = s[(6 * half + b) * stride + i];
+    } else if constexpr (P == 4) {
+        const float4 *s = reinterpret_cast<const float4 *>(in);
+        float4 *d = reinterpret_cast<float4 *>(dst);
+        for (int b = 0; b < 3; ++b) d[b * fstride + f] = s[(3 * half + b) * stride + i];
+    } else {
+        const short4 *s = reinterpret_cast<const short4 *>(in);
+        short4 *d = reinterpret_cast<short4 *>(dst);
+        for (int b = 0; b < 3; ++b) d[b * fstride + f] = s[(3 * half + b) * stride + i];
+        FaceIO<2>::norms(dst, fstride)[f] = SpinorIO<2>::norms(in, stride)[i];
+    }
+}
+
+void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back, void *send_fwd,
+                       cudaStream_t s) {
+    // non-dagger: the receiver's forward hop (1 - gamma_4) needs LOWER spins of our t=0 slice
+    // (sent backward); its backward hop (1 + gamma_4) needs UPPER spins of our t=T_loc-1 slice
+    // (sent forward).  The dagger swaps the halves (reading Q15).
+    const int half_back = dagger ? 0 : 1;
+    const int half_fwd = dagger ? 1 : 0;
+    const int T = 128;
+    const int b = nblk(2 * g.F, T);
+    if (prec == 8) k_pack_faces<8><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
+    else if (prec == 4) k_pack_faces<4><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
+    else k_pack_faces<2><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
+    QX_CUDA(cudaGetLastError());
+}
+
+}  // namespace qx

@@ -1,0 +1,218 @@
+// solver.cpp — mixed-precision BiCGstab with reliable updates (
+// BiCGstab: van der Vorst, ref [8]; reliable updates: Sleijpen & van der Vorst, ref [21]).
+//
+// "Algorithm R" (reading Q10): the Krylov iteration runs in the sloppy precision
+// on the even-odd operator Mhat; the solution accumulates in a sloppy xs that is folded into
+// the high-precision x at every reliable update, where the true residual r = bhat - Mhat x is
+// recomputed in the high precision.  One Krylov space is kept throughout (p, v continue across
+// updates).  The solve stops only on a TRUE residual <= tol ||bhat||.
+//
+//   setup: x = 0; r = bhat; rs = lo(r); rhat0 = rs; xs = 0; r0Norm = maxrr = maxrx = ||r||
+//   iterate:
+//     rho' = <rhat0, rs>;  p = rs (first) | rs + beta (p - omega v), beta = (rho'/rho)(alpha/omega)
+//     v = Mhat p;  alpha = rho' / <rhat0, v>;  rs -= alpha v
+//     t = Mhat rs; omega = <t, rs> / |t|^2
+//     xs += alpha p + omega rs;  rs -= omega t;  rNorm = |rs|
+//     maxrx = max(maxrx, rNorm); maxrr = max(maxrr, rNorm)
+//     updX = rNorm < delta r0Norm && r0Norm <= maxrx
+//     updR = (rNorm < delta maxrr && r0Norm <= maxrr) || updX || rNorm <= tol ||bhat||
+//     on updR: x += xs; xs = 0; r = bhat - Mhat x (high); rs = lo(r); rNorm = |r|; maxrr = rNorm;
+//              rho' = <rhat0, rs> recomputed for the replaced residual;
+//              if updX: r0Norm = maxrx = rNorm;  stop if rNorm <= tol ||bhat||
+#include <cmath>
+#include <complex>
+#include <cstring>
+
+#include "ctx.h"
+
+namespace qx {
+
+using cd = std::complex<double>;
+
+static void *field(qudax_ctx *c, void *&slot, int prec) {
+    if (!slot) slot = dalloc(c, spinor_bytes(prec, c->g.stride));
+    return slot;
+}
+
+static void zero(qudax_ctx *c, void *f, int prec) {
+    QX_CUDA(cudaMemsetAsync(f, 0, spinor_bytes(prec, c->g.stride), c->stream));
+}
+static void copy(qudax_ctx *c, void *dst, const void *src, int prec) {
+    QX_CUDA(cudaMemcpyAsync(dst, src, spinor_bytes(prec, c->g.stride), cudaMemcpyDeviceToDevice, c->stream));
+}
+
+static double norm2_of(qudax_ctx *c, int prec, void *f) {
+    double r;
+    void *fs[1] = {f};
+    blas_op(c, OP_NORM2, prec, fs, nullptr, &r);
+    return r;
+}
+static cd cdot_of(qudax_ctx *c, int prec, void *a, void *b) {
+    double r[2];
+    void *fs[2] = {a, b};
+    blas_op(c, OP_CDOT, prec, fs, nullptr, r);
+    return cd(r[0], r[1]);
+}
+
+void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *sp, qudax_solve_stats *st) {
+    QX_CHECK(c->gauge_loaded, QUDAX_ERR_STATE, "gauge not loaded");
+    const int Pd = sp->prec, Ps = sp->prec_sloppy;
+    check_prec(Pd);
+    check_prec(Ps);
+    QX_CHECK(sp->maxiter >= 0 && sp->tol >= 0 && sp->delta >= 0, QUDAX_ERR_ARG, "solve: bad parameters");
+    std::memset(st, 0, sizeof(*st));
+    auto &w = c->sws;
+    if (w.prec != Pd || w.prec_s != Ps) {
+        w = qudax_ctx::SolverWs{};  // (old buffers stay owned by the ctx until finalize)
+        w.prec = Pd;
+        w.prec_s = Ps;
+    }
+    const Geom &g = c->g;
+    const double kappa = c->kappa;
+    void *b_e = field(c, w.b_e, Pd), *b_o = field(c, w.b_o, Pd), *bh = field(c, w.bh, Pd);
+    void *x_e = field(c, w.x_e, Pd), *x_o = field(c, w.x_o, Pd), *r = field(c, w.r, Pd);
+    void *t_e = field(c, w.t_e, Pd), *t_o = field(c, w.t_o, Pd);
+    void *rs = field(c, w.rs, Ps), *xs = field(c, w.xs, Ps), *p = field(c, w.p, Ps);
+    void *v = field(c, w.v, Ps), *t = field(c, w.t, Ps), *r0 = field(c, w.r0, Ps);
+
+    // ---- load b (device fp64 DR slab) and prepare the Schur source
+    launch_spinor_import(Pd, g, 0, b_dev, b_e, c->stream);
+    launch_spinor_import(Pd, g, 1, b_dev, b_o, c->stream);
+    c->launches += 2;
+    if (sp->use_schur) {
+        clover_apply_op(c, t_o, b_o, Pd, 1, true);                // T_oo^{-1} b_o
+        dslash_op(c, t_e, t_o, nullptr, Pd, 0, 0, QUDAX_HOP, 0);  // D_eo T_oo^{-1} b_o
+        void *f[3] = {b_e, t_e, bh};
+        double a = kappa;
+        blas_op(c, OP_XPAY, Pd, f, &a, nullptr);                   // bhat = b_e + kappa (...)
+    } else {
+        copy(c, bh, b_e, Pd);
+    }
+
+    // ---- Algorithm R
+    const double b2 = norm2_of(c, Pd, bh);
+    const double bnorm = std::sqrt(b2);
+    const double stop = sp->tol * bnorm;
+    zero(c, x_e, Pd);
+    zero(c, xs, Ps);
+    zero(c, v, Ps);
+    zero(c, p, Ps);
+    copy(c, r, bh, Pd);
+    convert_op(c, rs, Ps, r, Pd);
+    copy(c, r0, rs, Ps);
+    double rNorm = bnorm;
+    double r0Norm = rNorm, maxrr = rNorm, maxrx = rNorm;
+    cd rho(1, 0), alpha(1, 0), omega(1, 0);
+    cd rho_new = cdot_of(c, Ps, r0, rs);
+    int k = 0, updates = 0;
+    bool converged = (bnorm == 0.0);
+    const double V_h_all = (double)g.Vh * g.nranks;
+    double flops = 0;
+    qudax_site_model mm;
+    qudax_model(4, 12, -1, &mm);  // 3696 flops / site for Mhat (precision independent)
+    const double matpc_flops = mm.flops * V_h_all;
+    const double blas_flops_iter = 960.0 * V_h_all;  // reading Q16 (fused BLAS per iteration)
+
+    while (!converged && k < sp->maxiter) {
+        if (k == 0) {
+            copy(c, p, rs, Ps);
+        } else {
+            cd beta = (rho_new / rho) * (alpha / omega);
+            void *f[3] = {rs, p, v};
+            double co[4] = {beta.real(), beta.imag(), omega.real(), omega.imag()};
+            blas_op(c, OP_P_UPDATE, Ps, f, co, nullptr);
+        }
+        matpc_op(c, v, p, Ps, 0);
+        cd r0v = cdot_of(c, Ps, r0, v);
+        alpha = rho_new / r0v;
+        {
+            void *f[2] = {v, rs};
+            double co[2] = {-alpha.real(), -alpha.imag()};
+            blas_op(c, OP_CAXPY, Ps, f, co, nullptr);
+        }
+        matpc_op(c, t, rs, Ps, 0);
+        double td[3];
+        {
+            void *f[2] = {t, rs};
+            blas_op(c, OP_TDOT, Ps, f, nullptr, td);
+        }
+        omega = cd(td[0], td[1]) / td[2];
+        double fin[3];
+        {
+            void *f[5] = {xs, p, rs, t, r0};
+            double co[4] = {alpha.real(), alpha.imag(), omega.real(), omega.imag()};
+            blas_op(c, OP_FINAL, Ps, f, co, fin);
+        }
+        rho = rho_new;
+        rho_new = cd(fin[1], fin[2]);
+        rNorm = std::sqrt(fin[0]);
+        ++k;
+        flops += 2 * matpc_flops + blas_flops_iter;
+        if (rNorm > maxrx) maxrx = rNorm;
+        if (rNorm > maxrr) maxrr = rNorm;
+        const bool updX = (rNorm < sp->delta * r0Norm) && (r0Norm <= maxrx);
+        const bool updR = ((rNorm < sp->delta * maxrr) && (r0Norm <= maxrr)) || updX || (rNorm <= stop) ||
+                          (k == sp->maxiter);
+        if (updR) {
+            xpy_mixed_op(c, Pd, Ps, xs, x_e);   // x += xs
+            zero(c, xs, Ps);
+            matpc_op(c, r, x_e, Pd, 0);          // r = Mhat x (high)
+            double r2;
+            {
+                void *f[2] = {bh, r};
+                blas_op(c, OP_BMR_NORM, Pd, f, nullptr, &r2);  // r = bhat - r
+            }
+            flops += matpc_flops;
+            convert_op(c, rs, Ps, r, Pd);
+            rNorm = std::sqrt(r2);
+            maxrr = rNorm;
+            if (updX) {
+                r0Norm = rNorm;
+                maxrx = rNorm;
+            }
+            rho_new = cdot_of(c, Ps, r0, rs);
+            ++updates;
+            if (rNorm <= stop) converged = true;
+        }
+    }
+    st->iters = k;
+    st->reliable_updates = updates;
+    st->true_res_schur = bnorm > 0 ? rNorm / bnorm : 0.0;
+
+    // ---- reconstruct the odd sites and the full-system true residual (fp64 if Pd == 8)
+    if (sp->use_schur) {
+        dslash_op(c, t_o, x_e, nullptr, Pd, 1, 0, QUDAX_HOP, 0);  // D_oe x_e
+        {
+            void *f[3] = {b_o, t_o, t_o};
+            double a = kappa;
+            blas_op(c, OP_XPAY, Pd, f, &a, nullptr);               // b_o + kappa D_oe x_e
+        }
+        clover_apply_op(c, x_o, t_o, Pd, 1, true);                 // x_o = T_oo^{-1}(...)
+        // (M x)_e = T_ee x_e - kappa D_eo x_o ; (M x)_o = T_oo x_o - kappa D_oe x_e
+        dslash_op(c, t_e, x_o, x_e, Pd, 0, 0, QUDAX_CLOVER_XPAY, -kappa);
+        dslash_op(c, t_o, x_e, x_o, Pd, 1, 0, QUDAX_CLOVER_XPAY, -kappa);
+        double re2, ro2;
+        {
+            void *f[2] = {b_e, t_e};
+            blas_op(c, OP_BMR_NORM, Pd, f, nullptr, &re2);
+        }
+        {
+            void *f[2] = {b_o, t_o};
+            blas_op(c, OP_BMR_NORM, Pd, f, nullptr, &ro2);
+        }
+        const double bb = norm2_of(c, Pd, b_e) + norm2_of(c, Pd, b_o);
+        st->true_res = bb > 0 ? std::sqrt((re2 + ro2) / bb) : 0.0;
+        launch_spinor_export(Pd, g, 0, x_e, x_dev, c->stream);
+        launch_spinor_export(Pd, g, 1, x_o, x_dev, c->stream);
+        c->launches += 2;
+    } else {
+        st->true_res = st->true_res_schur;
+        QX_CUDA(cudaMemsetAsync(x_dev, 0, sizeof(double) * 24 * g.V, c->stream));
+        launch_spinor_export(Pd, g, 0, x_e, x_dev, c->stream);
+        c->launches += 1;
+    }
+    QX_CUDA(cudaStreamSynchronize(c->stream));
+    st->flops = flops;
+}
+
+}  // namespace qx

@@ -1,0 +1,67 @@
+"""Mixed-precision reliable-update BiCGstab through the C-ABI,
+checked against the fp64 oracle: the oracle's own true residual of the GPU solution, the
+GPU-reported residual vs the oracle's (|diff| <= 1e-9), and the solution vs the oracle solve."""
+import numpy as np
+import pytest
+
+import oracle
+import qgen
+from paper_1011_0024_b200 import qudax
+
+pytestmark = pytest.mark.gpu
+
+DIMS = (8, 8, 8, 16)
+KAPPA, CSW = 0.124, 1.0
+
+
+@pytest.fixture(scope="module")
+def system():
+    U = qgen.gauge(DIMS, 1003, eps=0.1)  # weak field
+    wc = oracle.WilsonClover(U, KAPPA, CSW, -1.0)
+    return U, wc
+
+
+@pytest.mark.parametrize("mode", [
+    # (prec, recon, prec_sloppy, recon_sloppy, delta, tol)
+    (8, 18, 4, 12, 0.1, 1e-12),   # double-single (reading Q11)
+    (8, 18, 2, 12, 1e-2, 1e-12),  # double-half (P:787-790 delta = 1e-2)
+    (8, 12, 8, 12, 1e-5, 1e-12),  # uniform double (delta = 1e-5)
+    (4, 12, 2, 12, 0.1, 1e-6),    # single-half (delta = 1e-1), tol near fp32 floor
+])
+def test_solver_vs_oracle(torch_cuda, system, mode):
+    U, wc = system
+    prec, recon, ps, rs, delta, tol = mode
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=prec, recon=recon, prec_sloppy=ps, recon_sloppy=rs, t_boundary=-1)
+    for spin, colour in ((0, 0), (1, 2)):
+        b = qgen.point_source(DIMS, spin, colour)
+        x, st = ctx.solve(b, tol=tol, delta=delta, maxiter=5000, prec=prec, prec_sloppy=ps)
+        res_oracle = np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b)
+        print(mode, st["iters"], st["reliable_updates"], st["true_res"], res_oracle)
+        if prec == 8:
+            assert res_oracle <= tol * (1 + 1e-3) + 1e-15
+            assert abs(st["true_res"] - res_oracle) <= 1e-9
+        else:
+            assert res_oracle <= tol * 1.5
+        # solution vs oracle BiCGstab on the Schur system
+        bh = wc.prepare(b)
+        xe, _ = oracle.bicgstab(wc.matpc, bh, tol=1e-13, maxiter=5000)
+        xo = wc.reconstruct(xe, b)
+        assert np.linalg.norm(x - xo) / np.linalg.norm(xo) < (1e-9 if prec == 8 else 1e-4)
+    ctx.close()
+
+
+def test_solver_fixed_iterations_and_device_entry(torch_cuda, system):
+    import torch
+    U, wc = system
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+    b = qgen.spinor(DIMS, 77)
+    bd = torch.from_numpy(b.view(np.float64).copy()).cuda()
+    xd = torch.zeros_like(bd)
+    st = ctx.solve_dev(xd, bd, tol=0.0, delta=0.1, maxiter=7, prec=8, prec_sloppy=4, allow_not_converged=True)
+    assert st["iters"] == 7
+    x = xd.cpu().numpy().view(np.complex128).reshape(b.shape)
+    res = np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b)
+    assert abs(res - st["true_res"]) < 1e-9
+    ctx.close()

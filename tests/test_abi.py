@@ -1,0 +1,82 @@
+"""CPU-side checks of the C-ABI library: it loads, exports every symbol include/qudax.h
+declares, and its host-only bookkeeping (partition, work/traffic model) matches the paper."""
+import ctypes
+import os
+import re
+
+import pytest
+
+from paper_1011_0024_b200 import qudax
+from qtest_util import ROOT, read_golden
+
+
+def header_symbols():
+    src = open(os.path.join(ROOT, "include", "qudax.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(qudax_[a-z0-9_]+)\s*\(", src)) - {"qudax_exchange_fn", "qudax_allreduce_fn",
+                                                                          "qudax_alloc_fn", "qudax_free_fn"})
+
+
+def test_library_exports_every_header_symbol():
+    L = qudax.lib()
+    syms = header_symbols()
+    assert len(syms) >= 25
+    missing = [s for s in syms if not hasattr(L, s)]
+    assert not missing, missing
+    # the binding declares a signature for each of them
+    assert set(syms) == set(qudax.SIGNATURES), set(syms) ^ set(qudax.SIGNATURES)
+
+
+def test_abi_version_and_status_strings():
+    assert qudax.lib().qudax_abi_version() == 1
+    assert qudax.status_string(0) == "ok"
+    assert "unsupported" in qudax.status_string(5)
+
+
+def test_site_model_reproduces_paper_counts():
+    """Mhat costs 3696 flops per 2976 bytes in single precision (fp32, 2-row links)."""
+    _, kv = read_golden("paper_counts.txt")
+    m = qudax.site_model(4, 12, -1)
+    assert m["flops"] == kv["flops_per_site_matpc_fp32"]
+    assert m["bytes_paper"] == kv["bytes_per_site_matpc_fp32"]
+    # SURVEY 8(d) byte table (compulsory bytes per Dslash output site, clover fused)
+    expect = {(8, 18): 2112, (8, 12): 1728, (8, 8): 1472, (4, 18): 1056, (4, 12): 864, (4, 8): 736,
+              (2, 18): 544, (2, 12): 448, (2, 8): 384}
+    for (p, r), b in expect.items():
+        assert qudax.site_model(p, r, qudax.CLOVER_INV)["bytes_compulsory"] == b, (p, r)
+    assert qudax.site_model(4, 12, qudax.HOP)["flops"] == 1320
+    assert qudax.site_model(4, 12, qudax.CLOVER_INV)["flops"] == 1824
+    assert qudax.site_model(4, 12, qudax.CLOVER_XPAY)["flops"] == 1872
+
+
+def test_partition_info():
+    p = qudax.partition_info((32, 32, 32, 256), 8, 3)
+    assert p["T_loc"] == 32 and p["t0"] == 96
+    assert p["rank_fwd"] == 4 and p["rank_back"] == 2
+    assert p["V_s"] == 32 ** 3 and p["V_h"] == 32 ** 3 * 16 and p["face_sites"] == 32 ** 3 // 2
+    assert not p["applies_bc_fwd"] and not p["applies_bc_back"]
+    # face message sizes at 32^3 — 786,432 B fp32, 458,752 B half, 1,572,864 B fp64
+    assert p["face_bytes"] == {"single": 786432, "half": 458752, "double": 1572864}
+    p0 = qudax.partition_info((4, 4, 4, 8), 2, 0)
+    p1 = qudax.partition_info((4, 4, 4, 8), 2, 1)
+    assert p0["applies_bc_back"] and not p0["applies_bc_fwd"]
+    assert p1["applies_bc_fwd"] and not p1["applies_bc_back"]
+    one = qudax.partition_info((4, 4, 4, 8), 1, 0)
+    assert one["applies_bc_fwd"] and one["applies_bc_back"] and one["rank_fwd"] == 0
+    for bad in [((3, 4, 4, 8), 1, 0), ((4, 4, 4, 8), 3, 0), ((4, 4, 4, 6), 2, 0), ((4, 4, 4, 8), 8, 0),
+                ((4, 4, 4, 8), 2, 2)]:
+        with pytest.raises(qudax.QudaxError):
+            qudax.partition_info(*bad)
+
+
+def test_init_without_gpu_fails_loudly():
+    import torch
+    if torch.cuda.is_available():
+        pytest.skip("a GPU is present")
+    p = qudax.InitParam()
+    p.global_dims = (ctypes.c_int * 4)(4, 4, 4, 4)
+    p.nranks, p.rank, p.device, p.comm = 1, 0, 0, qudax.COMM_NONE
+    h = ctypes.c_void_p()
+    st = qudax.lib().qudax_init(ctypes.byref(h), ctypes.byref(p))
+    assert st == 3  # QUDAX_ERR_CUDA: no silent CPU fallback
+    assert not h.value
