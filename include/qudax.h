@@ -137,6 +137,9 @@ typedef struct {
     int prec_sloppy;             /* precision of the Krylov iteration (must have a gauge copy) */
     int prec;                    /* outer precision of x, r and the reliable-update residual */
     int use_schur;               /* 1: solve the full system M x = b via prepare/Mhat/reconstruct */
+    double *res_history;         /* optional host array: ||r_k|| / ||bhat|| after iteration k (the
+                                    iterated residual, replaced by the true one at reliable updates) */
+    int history_cap;             /* capacity of res_history (0 = none) */
 } qudax_solve_param;
 
 typedef struct {

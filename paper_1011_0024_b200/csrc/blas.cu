@@ -189,9 +189,7 @@ __global__ void k_bicg_final(long Vh, long stride, void *x, const void *p, void 
             ss[2 * k] = o.r;
             ss[2 * k + 1] = o.i;
         }
-        SpinorIO<P>::store(s, stride, i, ss);
-        // reduce what was stored (re-read is unnecessary for fp32/fp64; half uses the quantised value)
-        if constexpr (P == 2) SpinorIO<P>::load(s, stride, i, ss);
+        SpinorIO<P>::store_requant(s, stride, i, ss);  // reduce exactly what was stored
         R rh[24];
         SpinorIO<P>::load(rhat, stride, i, rh);
 #pragma unroll
@@ -228,11 +226,10 @@ __global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, double 
         SpinorIO<P>::load(b, stride, i, bb);
         SpinorIO<P>::load(r, stride, i, rr);
 #pragma unroll
-        for (int k = 0; k < 24; ++k) {
-            rr[k] = bb[k] - rr[k];
-            acc[0] += (double)rr[k] * rr[k];
-        }
-        SpinorIO<P>::store(r, stride, i, rr);
+        for (int k = 0; k < 24; ++k) rr[k] = bb[k] - rr[k];
+        SpinorIO<P>::store_requant(r, stride, i, rr);
+#pragma unroll
+        for (int k = 0; k < 24; ++k) acc[0] += (double)rr[k] * rr[k];
     }
     block_reduce_store<1>(acc, partials);
 }

@@ -188,6 +188,21 @@ struct SpinorIO {
             Blocks<P, 2 * BPH, false>::store(base, stride, i, 0, in);
         }
     }
+    // store, and replace `v` by exactly what a later load() of this site returns (half:
+    // the dequantised values) — lets a kernel reduce over what it stored without re-reading
+    // its own output through the non-coherent read-only path.
+    static __device__ __forceinline__ void store_requant(void *base, long stride, long i, R *v) {
+        store(base, stride, i, v);
+        if constexpr (P == 2) {
+            float m = 0.f;
+#pragma unroll
+            for (int k = 0; k < 24; ++k) m = fmaxf(m, fabsf(v[k]));
+            const float inv = (m > 0.f) ? kHalfMax / m : 0.f;
+            const float scale = m * kHalfInv;
+#pragma unroll
+            for (int k = 0; k < 24; ++k) v[k] = scale * (float)(short)__float2int_rn(v[k] * inv);
+        }
+    }
 };
 
 // A face (12 reals per site): fp64 6 double2, fp32 3 float4, half 3 short4 + float norm[fstride]

@@ -174,6 +174,7 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
             ++updates;
             if (rNorm <= stop) converged = true;
         }
+        if (sp->res_history && k - 1 < sp->history_cap) sp->res_history[k - 1] = bnorm > 0 ? rNorm / bnorm : 0.0;
     }
     st->iters = k;
     st->reliable_updates = updates;

@@ -57,7 +57,8 @@ class GaugeParam(ctypes.Structure):
 
 class SolveParam(ctypes.Structure):
     _fields_ = [("tol", ctypes.c_double), ("delta", ctypes.c_double), ("maxiter", ctypes.c_int),
-                ("prec_sloppy", ctypes.c_int), ("prec", ctypes.c_int), ("use_schur", ctypes.c_int)]
+                ("prec_sloppy", ctypes.c_int), ("prec", ctypes.c_int), ("use_schur", ctypes.c_int),
+                ("res_history", ctypes.POINTER(ctypes.c_double)), ("history_cap", ctypes.c_int)]
 
 
 class SolveStats(ctypes.Structure):
@@ -350,15 +351,21 @@ class Context:
         return complex(r[0], r[1])
 
     # -- solver
-    def _solve_param(self, tol, delta, maxiter, prec, prec_sloppy, use_schur):
-        return SolveParam(float(tol), float(delta), int(maxiter), int(prec_sloppy), int(prec), int(bool(use_schur)))
+    def _solve_param(self, tol, delta, maxiter, prec, prec_sloppy, use_schur, history=None):
+        sp = SolveParam(float(tol), float(delta), int(maxiter), int(prec_sloppy), int(prec), int(bool(use_schur)))
+        if history is not None:
+            assert history.dtype == np.float64 and history.flags.c_contiguous
+            sp.res_history = history.ctypes.data_as(_DP)
+            sp.history_cap = int(history.size)
+        return sp
 
     def solve(self, b, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
-              allow_not_converged=False):
-        """x = M^{-1} b (host arrays, full local slab, DR basis); returns (x, stats dict)."""
+              allow_not_converged=False, history=None):
+        """x = M^{-1} b (host arrays, full local slab, DR basis); returns (x, stats dict).
+        history: optional float64 numpy array receiving ||r_k||/||bhat|| per iteration."""
         b = np.ascontiguousarray(b, dtype=np.complex128)
         x = np.zeros_like(b)
-        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur)
+        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history)
         st = SolveStats()
         rc = lib().qudax_solve_bicgstab(self._h, _dptr(x), _dptr(b), ctypes.byref(sp), ctypes.byref(st))
         if rc and not (allow_not_converged and rc == 6):
@@ -366,10 +373,10 @@ class Context:
         return x, st.as_dict()
 
     def solve_dev(self, x, b, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
-                  allow_not_converged=False):
+                  allow_not_converged=False, history=None):
         """Device-resident variant: x, b are float64 CUDA tensors holding the full local slab
         (T_loc, Z, Y, X, 4, 3, 2)."""
-        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur)
+        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history)
         st = SolveStats()
         rc = lib().qudax_solve_bicgstab_dev(self._h, x.data_ptr(), b.data_ptr(), ctypes.byref(sp), ctypes.byref(st))
         if rc and not (allow_not_converged and rc == 6):

@@ -51,6 +51,21 @@ def test_solver_vs_oracle(torch_cuda, system, mode):
     ctx.close()
 
 
+def test_uniform_double_tracks_oracle_history(torch_cuda, system):
+    """Uniform fp64 with delta = 0 (no intermediate reliable updates) must follow the oracle's
+    textbook BiCGstab residual history: pins the alpha / beta / omega recurrences."""
+    U, wc = system
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18)
+    b = qgen.point_source(DIMS, 0, 0)
+    h = np.zeros(200)
+    ctx.solve(b, tol=1e-12, delta=0.0, maxiter=200, prec=8, prec_sloppy=8, history=h)
+    _, hist = oracle.bicgstab(wc.matpc, wc.prepare(b), tol=1e-12, maxiter=200)
+    hist = np.array(hist)
+    assert np.all(np.abs(h[:10] - hist[:10]) <= 1e-8 * hist[:10])
+    ctx.close()
+
+
 def test_solver_fixed_iterations_and_device_entry(torch_cuda, system):
     import torch
     U, wc = system
