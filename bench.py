@@ -1,0 +1,355 @@
+#!/usr/bin/env python
+"""Benchmark of the hot path (BASELINE.json metric: "Dslash GFLOPS & HBM GB/s per B200 at
+1/2/4/8 GPUs; mixed-prec solve time").
+
+Workload (BASELINE.json configs[4], the weak-scaling configuration that fits one GPU and is
+defined at every GPU count): 32^3 x 64 sites per GPU, global lattice 32^3 x (64 N),
+T-partitioned across N ranks.  Weak-field SU(3) gauge (eps = 0.1),
+kappa = 0.124, c_sw = 1.0, antiperiodic T.
+
+One STEP = one mixed-precision reliable-update BiCGstab solve of a fixed ITERS iterations
+(tol = 0, delta = 0.1; fp64 outer with fp64 18-real links, fp32 sloppy with 12-real links),
+through the C-ABI entry qudax_solve_bicgstab_dev: Schur prepare, ITERS x (2 Mhat = 4 Dslash
+kernels + 4 halo exchanges, 5 fused BLAS kernels, 3 global reductions), the fp64 reliable
+updates, reconstruction and the fp64 true residual — every row of SURVEY §8(a) except the
+once-per-configuration setup (gauge upload, clover build).  value = effective flops
+(P:755-758 convention: 3696 per even site per Mhat + 960 BLAS, reading Q16) of all ranks /
+max-over-ranks device time.
+
+Run:   python bench.py [--gpus N --steps K --warmup W]
+       torchrun --nproc-per-node N bench.py --gpus N ...
+       python bench.py --impl reference      (the fp64 CPU oracle on the host cores)
+"""
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import tempfile
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "Dslash GFLOPS & HBM GB/s per B200 at 1/2/4/8 GPUs; mixed-prec solve time"
+KAPPA, CSW, EPS = 0.124, 1.0, 0.1
+SPATIAL, T_PER_GPU = 32, 64
+GAUGE_SEED, SRC_SEED = 1005, 2005
+BLAS_FLOPS_PER_SITE_ITER = 960.0
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--iters", type=int, default=100, help="BiCGstab iterations per step")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-extra", action="store_true", help="skip the per-precision Dslash table and the config-3 solve")
+    ap.add_argument("--overlap", type=int, default=1)
+    return ap.parse_args()
+
+
+# ---------------------------------------------------------------------------- clocks
+class ClockSampler:
+    """nvidia-smi clocks and throttle reasons sampled every 200 ms during the timed region."""
+    FIELDS = "index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.hw_slowdown," \
+             "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown," \
+             "clocks_event_reasons.sw_power_cap"
+
+    def __init__(self, device):
+        self.device = device
+        self.proc = None
+        self.path = None
+
+    def __enter__(self):
+        try:
+            fd, self.path = tempfile.mkstemp(suffix=".csv")
+            os.close(fd)
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.device), f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
+                 "-lms", "200"], stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
+        except Exception:  # noqa: BLE001
+            self.proc = None
+        return self
+
+    def __exit__(self, *a):
+        if self.proc is not None:
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except Exception:  # noqa: BLE001
+                self.proc.kill()
+
+    def summary(self):
+        if not self.path or not os.path.exists(self.path):
+            return None
+        rows = []
+        for line in open(self.path):
+            parts = [p.strip() for p in line.split(",")]
+            if len(parts) < 8:
+                continue
+            try:
+                rows.append((float(parts[1]), float(parts[2]), parts[4:8]))
+            except ValueError:
+                continue
+        os.unlink(self.path)
+        if not rows:
+            return None
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[k] for _, _, r in rows for k in range(4) if r[k].lower() == "active"})
+        sm_max = max(r[1] for r in rows)
+        loaded = [r[0] for r in rows if r[0] > 0.3 * sm_max] or [r[0] for r in rows]
+        return {"sm_mhz": statistics.median(loaded), "sm_max_mhz": sm_max, "reasons": reasons, "samples": len(rows)}
+
+
+# ---------------------------------------------------------------------------- helpers
+def measured_peak():
+    path = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    try:
+        d = json.load(open(path))
+        return float(d["hbm_gbs"]), "MEASURED_PEAKS.json hbm_gbs (STREAM-style copy, of measured)"
+    except Exception:  # noqa: BLE001
+        return 6650.0, "B200_PROFILING.md fallback 6.65 TB/s (of fallback)"
+
+
+def profiled_traffic():
+    """dram bytes per Dslash launch from the committed ncu --set full summary (or None)."""
+    path = os.path.join(ROOT, "profiles", "dslash_traffic.json")
+    try:
+        d = json.load(open(path))
+        return d
+    except Exception:  # noqa: BLE001
+        return None
+
+
+def cpu_oracle_gflops(iters, dims=(SPATIAL, SPATIAL, SPATIAL, 8)):
+    """The fp64 oracle (oracle/, as it stands) on a bounded sample: `iters` textbook BiCGstab
+    iterations on Mhat of a 32^3 x 8 lattice of the same kind (weak field, same kappa/c_sw).
+    Returns (gflops, seconds, threads, sample description)."""
+    import numpy as np
+
+    import oracle
+    import qgen
+    U = qgen.gauge(dims, GAUGE_SEED, eps=EPS)
+    wc = oracle.WilsonClover(U, KAPPA, CSW, -1.0)
+    b = oracle.restrict(qgen.spinor(dims, SRC_SEED), 0)
+    t0 = time.perf_counter()
+    oracle.bicgstab(wc.matpc, b, tol=0.0, maxiter=iters)
+    dt = time.perf_counter() - t0
+    vh = np.prod(dims) / 2
+    flops = iters * (2 * 3696 + BLAS_FLOPS_PER_SITE_ITER) * vh
+    threads = int(os.environ.get("OMP_NUM_THREADS", os.cpu_count() or 1))
+    sample = f"{iters} oracle BiCGstab iterations on Mhat of a {dims[0]}^3x{dims[3]} weak-field lattice (fp64, C+OpenMP+numpy)"
+    return flops / dt * 1e-9, dt, threads, sample
+
+
+# ---------------------------------------------------------------------------- reference arm
+def run_reference(args):
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return
+    K, W = args.steps, args.warmup
+    iters = 2
+    for _ in range(W):
+        cpu_oracle_gflops(1)
+    times, gfl = [], []
+    for _ in range(K):
+        g, dt, threads, sample = cpu_oracle_gflops(iters)
+        times.append(dt)
+        gfl.append(g)
+    value = sum(gfl) / len(gfl)
+    out = {
+        "impl": "reference", "metric": METRIC, "value": value, "unit": "GFLOPS", "n_gpus": args.gpus,
+        "steps": K, "warmup": W, "ms_per_step": 1e3 * sum(times) / len(times), "higher_is_better": True,
+        "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": {"workload": "oracle sample of the weak-scaling 32^3x64-per-GPU BiCGstab workload",
+                   "sample": sample},
+        "cpu_baseline": {"value": value, "unit": "GFLOPS", "cores": threads, "kind": "oracle", "sample": sample},
+        "e2e": {"value": value, "unit": "GFLOPS", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(out))
+
+
+# ---------------------------------------------------------------------------- our arm
+def main():
+    args = parse()
+    if args.impl == "reference":
+        return run_reference(args)
+    import numpy as np
+    import torch
+    import torch.distributed as dist
+
+    import qgen
+    from paper_1011_0024_b200 import qudax
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    N = world
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=dev)
+    dims = (SPATIAL, SPATIAL, SPATIAL, T_PER_GPU * N)
+    T_loc = T_PER_GPU
+
+    def barrier():
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+
+    def max_over_ranks(v):
+        if world == 1:
+            return v
+        t = torch.tensor([v], dtype=torch.float64, device=dev)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        return float(t.item())
+
+    # ---- context + setup (once per configuration, not timed)
+    if world > 1:
+        obj = [qudax.nccl_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(obj, src=0)
+        ctx = qudax.Context(dims, nranks=N, rank=rank, device=local, comm=qudax.COMM_NCCL, nccl_id=obj[0],
+                            overlap=bool(args.overlap))
+    else:
+        ctx = qudax.Context(dims, device=local)
+    t0 = rank * T_loc
+    U = qgen.gauge(dims, GAUGE_SEED, eps=EPS, t_begin=t0, nt=T_loc)
+    ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12, t_boundary=-1)
+    del U
+    b_host = qgen.spinor(dims, SRC_SEED, t_begin=t0, nt=T_loc)
+    with torch.cuda.stream(ctx.stream):
+        b_dev = torch.from_numpy(b_host.view(np.float64)).to(dev)
+        x_dev = torch.zeros_like(b_dev)
+    ctx.stream.synchronize()
+    b_pin = torch.from_numpy(b_host.view(np.float64)).pin_memory()
+    x_pin = torch.zeros_like(b_pin).pin_memory()
+    solve_kw = dict(tol=0.0, delta=0.1, maxiter=args.iters, prec=8, prec_sloppy=4, allow_not_converged=True)
+
+    # ---- warm-up
+    for _ in range(args.warmup):
+        ctx.solve_dev(x_dev, b_dev, **solve_kw)
+    barrier()
+
+    # ---- timed region (device-resident inputs)
+    l0 = ctx.launch_count()
+    ctx.kernel_timing(True)
+    flops = 0.0
+    iters = 0
+    updates = 0
+    with ClockSampler(local) as clk:
+        barrier()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record(ctx.stream)
+        for _ in range(args.steps):
+            st = ctx.solve_dev(x_dev, b_dev, **solve_kw)
+            flops += st["flops"]
+            iters += st["iters"]
+            updates += st["reliable_updates"]
+        e1.record(ctx.stream)
+        barrier()
+    ms = max_over_ranks(e0.elapsed_time(e1))
+    launches = ctx.launch_count() - l0
+    ks = ctx.kernel_stats(prec=4)  # the sloppy fp32 recon-12 Dslash: the dominant kernel
+    ctx.kernel_timing(False)
+    clocks = clk.summary()
+    value = flops / (ms * 1e-3) * 1e-9  # flops already counts all ranks' sites
+
+    # ---- roofline of the dominant kernel (the Dslash, fp32 12-reconstruct, both kinds)
+    peak, peak_src = measured_peak()
+    avg_ms = ks["ms_total"] / max(ks["launches"], 1)
+    achieved = ks["bytes_compulsory"] / (ks["ms_total"] * 1e-3) * 1e-9 if ks["ms_total"] > 0 else 0.0
+    trafficd = profiled_traffic()
+    traffic = None
+    if trafficd and trafficd.get("lattice") == [SPATIAL, SPATIAL, SPATIAL, T_loc]:
+        traffic = trafficd.get("dram_bytes_per_launch")
+    roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
+                "traffic": traffic, "kernel": "dslash_kernel fp32 recon-12 (clover-inverse + clover-xpay kinds)",
+                "bytes_model": "compulsory (SURVEY 8(d)): 864 B/site clover-inv, 960 B/site xpay",
+                "avg_launch_ms": avg_ms, "launches": ks["launches"], "peak_source": peak_src,
+                "kernel_gflops": ks["flops"] / (ks["ms_total"] * 1e-3) * 1e-9 if ks["ms_total"] > 0 else 0.0,
+                "paper_model_gbs": ks["bytes_paper"] / (ks["ms_total"] * 1e-3) * 1e-9 if ks["ms_total"] > 0 else 0.0,
+                "kernel_share_of_step": ks["ms_total"] / ms if ms > 0 else None}
+
+    # ---- end to end through the C-ABI with pinned host buffers (H2D of b, D2H of x inside)
+    barrier()
+    e2 = [torch.cuda.Event(enable_timing=True) for _ in range(2)]
+    flops_e2e = 0.0
+    e2[0].record(ctx.stream)
+    for _ in range(args.steps):
+        _, st = ctx.solve(b_pin, out=x_pin, **solve_kw)
+        flops_e2e += st["flops"]
+    e2[1].record(ctx.stream)
+    barrier()
+    ms_e2e = max_over_ranks(e2[0].elapsed_time(e2[1]))
+    nbytes = b_pin.numel() * 8
+    e2e = {"value": flops_e2e / (ms_e2e * 1e-3) * 1e-9, "unit": "GFLOPS", "h2d_bytes_per_step": nbytes,
+           "d2h_bytes_per_step": nbytes, "api": "qudax_solve_bicgstab (host buffers, pinned)"}
+
+    # ---- Dslash-only numbers (Mhat applications, device resident), per precision
+    dslash = {}
+    if not args.no_extra:
+        for prec, recon, name in ((4, 12, "fp32-12"), (8, 18, "fp64-18")):
+            fin, fout = ctx.new_field(prec), ctx.new_field(prec)
+            ctx.spinor_load_dev(fin, prec, 0, b_dev)
+            for _ in range(5):
+                ctx.matpc(fout, fin, prec)
+            barrier()
+            ctx.kernel_timing(True)
+            ea, eb = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            reps = 50
+            ea.record(ctx.stream)
+            for _ in range(reps):
+                ctx.matpc(fout, fin, prec)
+            eb.record(ctx.stream)
+            barrier()
+            mms = max_over_ranks(ea.elapsed_time(eb))
+            k2 = ctx.kernel_stats(prec=prec)
+            ctx.kernel_timing(False)
+            m = qudax.site_model(prec, recon, -1)
+            sites = (SPATIAL ** 3 * T_loc // 2) * N
+            per_gpu = sites / N * reps
+            dslash[name] = {
+                "matpc_gflops_total": m["flops"] * sites * reps / (mms * 1e-3) * 1e-9,
+                "matpc_gflops_per_gpu": m["flops"] * per_gpu / (mms * 1e-3) * 1e-9,
+                "matpc_us": 1e3 * mms / reps,
+                "model_gbs_per_gpu": m["bytes_compulsory"] * per_gpu / (mms * 1e-3) * 1e-9,
+                "kernel_gbs_compulsory": k2["bytes_compulsory"] / (k2["ms_total"] * 1e-3) * 1e-9,
+                "kernel_gflops": k2["flops"] / (k2["ms_total"] * 1e-3) * 1e-9,
+                "frac_of_measured_hbm": (k2["bytes_compulsory"] / (k2["ms_total"] * 1e-3) * 1e-9) / peak,
+            }
+            del fin, fout
+
+    # ---- CPU baseline: the oracle on the host cores (rank 0, N = 1 only)
+    cpu = None
+    if rank == 0 and N == 1 and not args.no_cpu_baseline:
+        g, dt, threads, sample = cpu_oracle_gflops(6)
+        cpu = {"value": g, "unit": "GFLOPS", "cores": threads, "kind": "oracle", "sample": sample, "seconds": dt}
+
+    ctx.close()
+    if rank == 0:
+        out = {
+            "metric": METRIC, "value": value, "unit": "GFLOPS", "n_gpus": N, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": ms / args.steps, "higher_is_better": True, "scaling": "weak",
+            "vs_baseline": None, "dtype": "f32", "data": "synthetic",
+            "config": {"workload": f"weak scaling 32^3x64 per GPU (global 32^3x{T_PER_GPU * N}), mixed-precision "
+                                   f"reliable-update BiCGstab, {args.iters} iterations per step (BASELINE configs[4])",
+                       "lattice_global": list(dims), "lattice_per_gpu": [SPATIAL, SPATIAL, SPATIAL, T_loc],
+                       "precision": {"outer": "f64 recon-18", "sloppy": "f32 recon-12"},
+                       "kappa": KAPPA, "csw": CSW, "gauge": f"weak field eps={EPS}", "t_boundary": "antiperiodic",
+                       "delta": 0.1, "parallelism": f"T-slab x{N}" + (" (NCCL halo, overlapped)" if N > 1 else ""),
+                       "l2": "inputs larger than L2 (>1 GB of gauge+clover+fields per GPU vs 126 MB L2)"},
+            "iters_per_step": iters / args.steps, "reliable_updates_per_step": updates / args.steps,
+            "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches, "clocks": clocks,
+            "dslash": dslash,
+        }
+        print(json.dumps(out))
+    if world > 1:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

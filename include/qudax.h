@@ -167,6 +167,16 @@ typedef struct {
                                     half including its per-site norms */
 } qudax_partition;
 
+/* Accumulated CUDA-event timing of the Dslash kernel launches since qudax_kernel_timing(ctx, 1). */
+typedef struct {
+    long long launches;          /* Dslash kernel launches recorded (interior + boundary count separately) */
+    long long sites;             /* output sites processed by them */
+    double ms_total;             /* sum of per-launch durations (events on the launching stream) */
+    double flops;                /* effective flops of those launches (qudax_model per kind) */
+    double bytes_compulsory;     /* algorithmic bytes (compulsory model) of those launches */
+    double bytes_paper;          /* paper-model bytes */
+} qudax_kernel_stats;
+
 /* ---- host-only helpers (no GPU needed) ---- */
 int qudax_abi_version(void);
 const char *qudax_status_string(int status);
@@ -186,6 +196,10 @@ qudax_status qudax_sync(qudax_ctx *ctx);
 /* Number of library kernels launched by this ctx so far (for launch accounting). */
 long long qudax_launch_count(const qudax_ctx *ctx);
 qudax_status qudax_get_partition(const qudax_ctx *ctx, qudax_partition *out);
+/* Enable (1) / disable (0) per-launch event timing of the Dslash kernels; clears the records. */
+qudax_status qudax_kernel_timing(qudax_ctx *ctx, int enable);
+/* Synchronise and sum the recorded Dslash launches of precision prec_filter (0 = all). */
+qudax_status qudax_get_kernel_stats(qudax_ctx *ctx, int prec_filter, qudax_kernel_stats *out);
 
 /* ---- gauge field and clover (setup) ----
  * Uploads the host slab, exchanges the gauge ghost / clover halo timeslices with the T

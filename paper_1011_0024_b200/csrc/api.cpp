@@ -113,11 +113,36 @@ static void exchange(qudax_ctx *c, const void *send_fwd, const void *send_back, 
     }
 }
 
-static void launch_dslash_any(int prec, int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
+static cudaEvent_t pool_event(qudax_ctx *c) {
+    if (!c->ev_pool.empty()) {
+        cudaEvent_t e = c->ev_pool.back();
+        c->ev_pool.pop_back();
+        return e;
+    }
+    cudaEvent_t e;
+    QX_CUDA(cudaEventCreate(&e));
+    return e;
+}
+
+static void launch_dslash_raw(int prec, int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
     if (prec == 8) launch_dslash_f64(recon, dagger, kind, a, s);
     else if (prec == 4) launch_dslash_f32(recon, dagger, kind, a, s);
     else launch_dslash_f16(recon, dagger, kind, a, s);
     QX_CUDA(cudaGetLastError());
+}
+
+// every Dslash kernel launch goes through here; with timing enabled it is bracketed by CUDA
+// events on the launching (compute) stream
+static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int kind, const DslashArgs &a) {
+    if (!c->timing) {
+        launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
+        return;
+    }
+    qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads};
+    QX_CUDA(cudaEventRecord(r.a, c->stream));
+    launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
+    QX_CUDA(cudaEventRecord(r.b, c->stream));
+    c->trecs.push_back(r);
 }
 
 void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
@@ -150,7 +175,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         args.ghosted = 0;
         args.range = RANGE_ALL;
         args.nthreads = (int)g.Vh;
-        launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+        launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
         c->launches += 1;
         return;
     }
@@ -169,17 +194,17 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         if (c->overlap && g.T_loc > 2) {
             args.range = RANGE_INTERIOR;
             args.nthreads = (int)((g.T_loc - 2) * g.F);
-            launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+            launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
             args.range = RANGE_BOUNDARY;
             args.nthreads = (int)(2 * g.F);
-            launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+            launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
             c->launches += 2;
         } else {
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
             args.range = RANGE_ALL;
             args.nthreads = (int)g.Vh;
-            launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+            launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
             c->launches += 1;
         }
     } else {  // HOST: paper strategy 1 (no overlap)
@@ -187,7 +212,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         exchange(c, h.sf, h.sb, h.gb, h.gf, h.bytes, c->stream, h.h_sf, h.h_sb, h.h_gb, h.h_gf);
         args.range = RANGE_ALL;
         args.nthreads = (int)g.Vh;
-        launch_dslash_any(prec, gc.recon, dagger, kind, args, c->stream);
+        launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
         c->launches += 2;
     }
 }
@@ -525,6 +550,8 @@ qudax_status qudax_finalize(qudax_ctx *c) {
         else cudaFree(p);
     }
     for (void *p : c->host_allocs) cudaFreeHost(p);
+    for (auto &r : c->trecs) { cudaEventDestroy(r.a); cudaEventDestroy(r.b); }
+    for (auto e : c->ev_pool) cudaEventDestroy(e);
     if (c->ev_in) cudaEventDestroy(c->ev_in);
     if (c->ev_halo) cudaEventDestroy(c->ev_halo);
     if (c->comm_stream) cudaStreamDestroy(c->comm_stream);
@@ -549,6 +576,40 @@ qudax_status qudax_get_partition(const qudax_ctx *c, qudax_partition *out) {
     if (!c || !out) return QUDAX_ERR_ARG;
     const int gd[4] = {c->g.X, c->g.Y, c->g.Z, c->g.T};
     return fill_partition(gd, c->g.nranks, c->g.rank, out);
+}
+
+qudax_status qudax_kernel_timing(qudax_ctx *c, int enable) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        for (auto &r : c->trecs) {
+            c->ev_pool.push_back(r.a);
+            c->ev_pool.push_back(r.b);
+        }
+        c->trecs.clear();
+        c->timing = enable != 0;
+    });
+}
+
+qudax_status qudax_get_kernel_stats(qudax_ctx *c, int prec_filter, qudax_kernel_stats *o) {
+    if (!c || !o) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        std::memset(o, 0, sizeof(*o));
+        for (auto &r : c->trecs) {
+            if (prec_filter && r.prec != prec_filter) continue;
+            float ms = 0;
+            QX_CUDA(cudaEventElapsedTime(&ms, r.a, r.b));
+            qudax_site_model m;
+            qudax_model(r.prec, r.recon, r.kind, &m);
+            o->launches += 1;
+            o->ms_total += ms;
+            o->sites += r.sites;
+            o->flops += m.flops * r.sites;
+            o->bytes_compulsory += m.bytes_compulsory * r.sites;
+            o->bytes_paper += m.bytes_paper * r.sites;
+        }
+    });
 }
 
 qudax_status qudax_gauge_load(qudax_ctx *c, const double *host_gauge, const qudax_gauge_param *p) {

@@ -26,6 +26,15 @@ struct qudax_ctx {
     std::string err;
     bool sticky = false;
     long long launches = 0;
+    // optional per-launch CUDA-event timing of the Dslash kernels (qudax_kernel_timing)
+    bool timing = false;
+    struct TimingRec {
+        cudaEvent_t a, b;
+        int prec, recon, kind;
+        long sites;
+    };
+    std::vector<TimingRec> trecs;
+    std::vector<cudaEvent_t> ev_pool;
     std::vector<void *> allocs;       // device allocations owned by the ctx
     std::vector<void *> host_allocs;  // pinned host allocations
 

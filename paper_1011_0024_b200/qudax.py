@@ -74,6 +74,14 @@ class SiteModel(ctypes.Structure):
     _fields_ = [("flops", ctypes.c_double), ("bytes_paper", ctypes.c_double), ("bytes_compulsory", ctypes.c_double)]
 
 
+class KernelStats(ctypes.Structure):
+    _fields_ = [("launches", ctypes.c_longlong), ("sites", ctypes.c_longlong), ("ms_total", ctypes.c_double),
+                ("flops", ctypes.c_double), ("bytes_compulsory", ctypes.c_double), ("bytes_paper", ctypes.c_double)]
+
+    def as_dict(self):
+        return {k: getattr(self, k) for k, _ in self._fields_}
+
+
 class Partition(ctypes.Structure):
     _fields_ = [("T_loc", ctypes.c_int), ("t0", ctypes.c_int), ("rank_fwd", ctypes.c_int),
                 ("rank_back", ctypes.c_int), ("V_loc", ctypes.c_long), ("V_h", ctypes.c_long),
@@ -103,6 +111,8 @@ SIGNATURES = {
     "qudax_sync": ([_P], _I),
     "qudax_launch_count": ([_P], ctypes.c_longlong),
     "qudax_get_partition": ([_P, ctypes.POINTER(Partition)], _I),
+    "qudax_kernel_timing": ([_P, _I], _I),
+    "qudax_get_kernel_stats": ([_P, _I, ctypes.POINTER(KernelStats)], _I),
     "qudax_gauge_load": ([_P, _DP, ctypes.POINTER(GaugeParam)], _I),
     "qudax_spinor_bytes": ([_P, _I], _Z),
     "qudax_spinor_load": ([_P, _P, _I, _I, _DP], _I),
@@ -226,7 +236,9 @@ class Context:
         self.global_dims = tuple(int(d) for d in global_dims)
         self.device = int(device)
         torch.cuda.set_device(self.device)
-        self.stream = stream if stream is not None else torch.cuda.current_stream(self.device)
+        # the library's compute stream: a dedicated torch stream unless the caller passes one;
+        # record events / order torch work against ctx.stream
+        self.stream = stream if stream is not None else torch.cuda.Stream(self.device)
         p = InitParam()
         p.global_dims = (ctypes.c_int * 4)(*self.global_dims)
         p.nranks, p.rank, p.device, p.comm, p.overlap = int(nranks), int(rank), self.device, int(comm), int(bool(overlap))
@@ -289,6 +301,14 @@ class Context:
     def sync(self):
         self._check(lib().qudax_sync(self._h))
 
+    def kernel_timing(self, enable=True):
+        self._check(lib().qudax_kernel_timing(self._h, int(bool(enable))))
+
+    def kernel_stats(self, prec=0):
+        out = KernelStats()
+        self._check(lib().qudax_get_kernel_stats(self._h, int(prec), ctypes.byref(out)))
+        return out.as_dict()
+
     # -- gauge
     def gauge_load(self, U, kappa, csw, prec=SINGLE, recon=12, prec_sloppy=None, recon_sloppy=None, t_boundary=-1):
         U = np.ascontiguousarray(U, dtype=np.complex128)
@@ -304,7 +324,9 @@ class Context:
         return int(lib().qudax_spinor_bytes(self._h, int(prec)))
 
     def new_field(self, prec):
-        return self._torch.zeros(self.spinor_bytes(prec), dtype=self._torch.uint8, device=f"cuda:{self.device}")
+        """A zeroed parity field, allocated and cleared on the library stream."""
+        with self._torch.cuda.stream(self.stream):
+            return self._torch.zeros(self.spinor_bytes(prec), dtype=self._torch.uint8, device=f"cuda:{self.device}")
 
     def spinor_load(self, field, prec, parity, psi):
         psi = np.ascontiguousarray(psi, dtype=np.complex128)
@@ -360,14 +382,19 @@ class Context:
         return sp
 
     def solve(self, b, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
-              allow_not_converged=False, history=None):
+              allow_not_converged=False, history=None, out=None):
         """x = M^{-1} b (host arrays, full local slab, DR basis); returns (x, stats dict).
         history: optional float64 numpy array receiving ||r_k||/||bhat|| per iteration."""
-        b = np.ascontiguousarray(b, dtype=np.complex128)
-        x = np.zeros_like(b)
+        if hasattr(b, "data_ptr"):  # torch CPU tensors (e.g. pinned float64 buffers), x preallocated
+            bp, x = ctypes.cast(b.data_ptr(), _DP), (out if out is not None else self._torch.zeros_like(b))
+            xp = ctypes.cast(x.data_ptr(), _DP)
+        else:
+            b = np.ascontiguousarray(b, dtype=np.complex128)
+            x = np.zeros_like(b) if out is None else out
+            bp, xp = _dptr(b), _dptr(x)
         sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history)
         st = SolveStats()
-        rc = lib().qudax_solve_bicgstab(self._h, _dptr(x), _dptr(b), ctypes.byref(sp), ctypes.byref(st))
+        rc = lib().qudax_solve_bicgstab(self._h, xp, bp, ctypes.byref(sp), ctypes.byref(st))
         if rc and not (allow_not_converged and rc == 6):
             self._check(rc)
         return x, st.as_dict()
