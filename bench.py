@@ -326,7 +326,7 @@ def main():
     # ---- CPU baseline: the oracle on the host cores (rank 0, N = 1 only)
     cpu = None
     if rank == 0 and N == 1 and not args.no_cpu_baseline:
-        g, dt, threads, sample = cpu_oracle_gflops(6)
+        g, dt, threads, sample = cpu_oracle_gflops(20)
         cpu = {"value": g, "unit": "GFLOPS", "cores": threads, "kind": "oracle", "sample": sample, "seconds": dt}
 
     ctx.close()

@@ -57,6 +57,9 @@ def _load():
         _lib.oracle_invert12.argtypes = [dp, dp, ctypes.c_long]
         _lib.oracle_invert12.restype = ctypes.c_int
         _lib.oracle_site_mult.argtypes = [dp, dp, dp, ctypes.c_long]
+        lp = ctypes.POINTER(ctypes.c_long)
+        _lib.oracle_dslash_sites.argtypes = [dp, dp, dp, ip, ctypes.c_double, ctypes.c_int, lp, ctypes.c_long]
+        _lib.oracle_clover_sites.argtypes = [dp, dp, ip, ctypes.c_double, ctypes.c_double, lp, ctypes.c_long]
     return _lib
 
 
@@ -196,6 +199,81 @@ class WilsonClover:
         b_o = restrict(b, 1)
         x_o = self.Tinv_pp(b_o + self.kappa * self.Dpq(x_e, 1), 1)
         return x_e + x_o
+
+
+# ----------------------------------------------------------------------------- sampled sites
+# For lattices too large to evaluate everywhere (BASELINE full sizes), the same per-site
+# arithmetic as dslash()/clover() (oracle.c: dslash_one / clover_one) evaluated at a list of
+# lexicographic site indices of the global lattice.
+
+def _sites_arr(sites):
+    s = np.ascontiguousarray(np.asarray(sites, dtype=np.int64))
+    return s, s.ctypes.data_as(ctypes.POINTER(ctypes.c_long))
+
+
+def dslash_sites(U, psi, sites, t_bc=-1.0, dagger=False):
+    """(D psi)(x) for x in sites; returns [len(sites), 4, 3]."""
+    dims = _dims_of_spinor(psi)
+    s, sp = _sites_arr(sites)
+    out = np.empty((len(s), 4, 3), dtype=np.complex128)
+    _load().oracle_dslash_sites(_p(out), _p(np.ascontiguousarray(U)), _p(np.ascontiguousarray(psi)), _cdims(dims),
+                                float(t_bc), int(bool(dagger)), sp, len(s))
+    return out
+
+
+def clover_sites(U, sites, kappa, csw):
+    T_, Z, Y, X = U.shape[1:5]
+    s, sp = _sites_arr(sites)
+    out = np.empty((len(s), 12, 12), dtype=np.complex128)
+    _load().oracle_clover_sites(_p(out), _p(np.ascontiguousarray(U)), _cdims((X, Y, Z, T_)), float(kappa),
+                                float(csw), sp, len(s))
+    return out
+
+
+def neighbours(dims, sites):
+    """The 8 nearest neighbours (lex indices) of each site, shape [n, 8]."""
+    X, Y, Z, T = dims
+    s = np.asarray(sites, dtype=np.int64)
+    c = [s % X, (s // X) % Y, (s // (X * Y)) % Z, s // (X * Y * Z)]
+    L = [X, Y, Z, T]
+    out = []
+    for mu in range(4):
+        for step in (1, -1):
+            n = [ci.copy() for ci in c]
+            n[mu] = (n[mu] + step) % L[mu]
+            out.append(((n[3] * Z + n[2]) * Y + n[1]) * X + n[0])
+    return np.stack(out, axis=1)
+
+
+def apply_M_chunked(U, x, kappa, csw, t_bc=-1.0, chunk=1 << 17):
+    """M_kappa x = T x - kappa D x on the whole lattice without storing the 12x12 clover of
+    every site (T is evaluated chunk by chunk with clover_sites): for full-size residuals."""
+    dims = _dims_of_spinor(x)
+    out = -kappa * dslash(U, x, t_bc)
+    xf = x.reshape(-1, 12)
+    of = out.reshape(-1, 12)
+    V = xf.shape[0]
+    for s0 in range(0, V, chunk):
+        idx = np.arange(s0, min(V, s0 + chunk))
+        of[idx] += np.einsum("nij,nj->ni", clover_sites(U, idx, kappa, csw), xf[idx])
+    return out
+
+
+def matpc_sites(U, psi_e, sites, kappa, csw, t_bc=-1.0, dagger=False):
+    """(Mhat psi_e)(x) for even sites x, Mhat = T_ee - kappa^2 D_eo T_oo^{-1} D_oe, evaluated
+    only where needed: D_oe psi_e at the odd neighbours of the sample, T^{-1} there, then D_eo at
+    the sample.  psi_e: full-lattice array zero on odd sites."""
+    dims = _dims_of_spinor(psi_e)
+    sites = np.asarray(sites, dtype=np.int64)
+    nb = np.unique(neighbours(dims, sites).ravel())
+    d_nb = dslash_sites(U, psi_e, nb, t_bc, dagger)
+    tinv = invert12(clover_sites(U, nb, kappa, csw))
+    tmp = np.zeros_like(psi_e)
+    tmp.reshape(-1, 4, 3)[nb] = np.einsum("nij,nj->ni", tinv, d_nb.reshape(-1, 12)).reshape(-1, 4, 3)
+    dd = dslash_sites(U, tmp, sites, t_bc, dagger)
+    Tx = clover_sites(U, sites, kappa, csw)
+    tx = np.einsum("nij,nj->ni", Tx, psi_e.reshape(-1, 12)[sites]).reshape(-1, 4, 3)
+    return tx - kappa ** 2 * dd
 
 
 # ----------------------------------------------------------------------------- solver

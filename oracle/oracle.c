@@ -74,18 +74,14 @@ static inline long neighbour(const long c[4], int mu, int step, const int d[4]) 
  * forward hop out of global t = T_global-1 and the backward hop out of global t = 0.
  * For the plain global lattice: t_global_offset = 0, T_global = dims[3].
  */
-void oracle_dslash(double *out_, const double *U_, const double *in_, const int dims[4],
-                   double t_bc, int dagger, int t_global_offset, int T_global) {
-    cplx *out = (cplx *)out_;
-    const cplx *U = (const cplx *)U_;
-    const cplx *in = (const cplx *)in_;
-    const long V = (long)dims[0] * dims[1] * dims[2] * dims[3];
+/* (D in)(x) or (D^dag in)(x) at the single site s, written to out[12] */
+static void dslash_one(cplx *out, long s, const cplx *U, const cplx *in, const int dims[4], long V, double t_bc,
+                       int dagger, int t_global_offset, int T_global) {
     /* non-dagger: forward hop (x+mu) uses (1 - gamma_mu), backward (x-mu) uses (1 + gamma_mu);
        the explicit adjoint swaps them. */
     const double sf = dagger ? +1.0 : -1.0;
     const double sb = -sf;
-#pragma omp parallel for schedule(static)
-    for (long s = 0; s < V; ++s) {
+    {
         long c[4];
         c[0] = s % dims[0];
         c[1] = (s / dims[0]) % dims[1];
@@ -136,8 +132,29 @@ void oracle_dslash(double *out_, const double *U_, const double *in_, const int 
                     }
             }
         }
-        memcpy(out + s * 12, acc, sizeof(acc));
+        memcpy(out, acc, sizeof(acc));
     }
+}
+
+void oracle_dslash(double *out_, const double *U_, const double *in_, const int dims[4],
+                   double t_bc, int dagger, int t_global_offset, int T_global) {
+    cplx *out = (cplx *)out_;
+    const long V = (long)dims[0] * dims[1] * dims[2] * dims[3];
+#pragma omp parallel for schedule(static)
+    for (long s = 0; s < V; ++s)
+        dslash_one(out + s * 12, s, (const cplx *)U_, (const cplx *)in_, dims, V, t_bc, dagger, t_global_offset,
+                   T_global);
+}
+
+/* The same operator evaluated only at the listed sites: out[k] = (D in)(sites[k]).  Used to
+ * check full-size GPU results on a sample of output sites. */
+void oracle_dslash_sites(double *out_, const double *U_, const double *in_, const int dims[4], double t_bc,
+                         int dagger, const long *sites, long nsites) {
+    cplx *out = (cplx *)out_;
+    const long V = (long)dims[0] * dims[1] * dims[2] * dims[3];
+#pragma omp parallel for schedule(static)
+    for (long k = 0; k < nsites; ++k)
+        dslash_one(out + k * 12, sites[k], (const cplx *)U_, (const cplx *)in_, dims, V, t_bc, dagger, 0, dims[3]);
 }
 
 /* 3x3 helpers */
@@ -174,12 +191,8 @@ static long shift2(const long c[4], int mu, int dmu, int nu, int dnu, const int 
  * Array treated periodic (gauge links carry no fermion boundary phase).
  * Out: Tout[lex][12][12] complex.
  */
-void oracle_clover(double *Tout_, const double *U_, const int dims[4], double kappa, double csw) {
-    cplx *Tout = (cplx *)Tout_;
-    const cplx *U = (const cplx *)U_;
-    const long V = (long)dims[0] * dims[1] * dims[2] * dims[3];
-#pragma omp parallel for schedule(static)
-    for (long s = 0; s < V; ++s) {
+static void clover_one(cplx *Tout, long s, const cplx *U, const int dims[4], long V, double kappa, double csw) {
+    {
         long c[4];
         c[0] = s % dims[0];
         c[1] = (s / dims[0]) % dims[1];
@@ -244,8 +257,24 @@ void oracle_clover(double *Tout_, const double *U_, const int dims[4], double ka
                         for (int a = 0; a < 3; ++a)
                             for (int b = 0; b < 3; ++b) T[r * 3 + a][q * 3 + b] += coef * gg[r][q] * F[a * 3 + b];
             }
-        memcpy(Tout + s * 144, T, sizeof(T));
+        memcpy(Tout, T, sizeof(T));
     }
+}
+
+void oracle_clover(double *Tout_, const double *U_, const int dims[4], double kappa, double csw) {
+    cplx *Tout = (cplx *)Tout_;
+    const long V = (long)dims[0] * dims[1] * dims[2] * dims[3];
+#pragma omp parallel for schedule(static)
+    for (long s = 0; s < V; ++s) clover_one(Tout + s * 144, s, (const cplx *)U_, dims, V, kappa, csw);
+}
+
+/* T at the listed sites only: Tout[k] = T(sites[k]). */
+void oracle_clover_sites(double *Tout_, const double *U_, const int dims[4], double kappa, double csw,
+                         const long *sites, long nsites) {
+    cplx *Tout = (cplx *)Tout_;
+    const long V = (long)dims[0] * dims[1] * dims[2] * dims[3];
+#pragma omp parallel for schedule(static)
+    for (long k = 0; k < nsites; ++k) clover_one(Tout + k * 144, sites[k], (const cplx *)U_, dims, V, kappa, csw);
 }
 
 /* Tinv(x) = T(x)^{-1} by Gauss-Jordan elimination with partial pivoting.

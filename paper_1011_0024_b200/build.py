@@ -36,13 +36,19 @@ def _needs(obj, deps):
     return any(os.path.getmtime(d) > t for d in deps)
 
 
-def build(force=False, verbose=False):
+def build(force=False, verbose=False, out_dir=None, defines=()):
+    """Compile and link libqudax.so.  out_dir/defines build experiment variants elsewhere
+    (e.g. -DQX_DSLASH_MINB=6); the product library is the default one in lib/."""
+    global OUT_DIR, LIB
+    if out_dir is not None:
+        OUT_DIR, LIB = out_dir, os.path.join(out_dir, "libqudax.so")
     inc, lib = nccl_dirs()
     os.makedirs(os.path.join(OUT_DIR, "obj"), exist_ok=True)
     headers = glob.glob(os.path.join(CSRC, "*.h")) + glob.glob(os.path.join(CSRC, "*.cuh")) + \
         [os.path.join(ROOT, "include", "qudax.h")]
     srcs = sorted(glob.glob(os.path.join(CSRC, "*.cu")) + glob.glob(os.path.join(CSRC, "*.cpp")))
     common = ["-O3", "-std=c++17", "-Xcompiler", "-fPIC", "-I", os.path.join(ROOT, "include"), "-I", CSRC, "-I", inc]
+    common += [f"-D{d}" for d in defines]
     jobs = []
     objs = []
     for s in srcs:
@@ -74,4 +80,6 @@ def build(force=False, verbose=False):
 
 
 if __name__ == "__main__":
-    print(build(force="--force" in sys.argv, verbose="-v" in sys.argv))
+    defs = [a[2:] for a in sys.argv[1:] if a.startswith("-D")]
+    od = next((a.split("=", 1)[1] for a in sys.argv[1:] if a.startswith("--out=")), None)
+    print(build(force="--force" in sys.argv, verbose="-v" in sys.argv, out_dir=od, defines=defs))

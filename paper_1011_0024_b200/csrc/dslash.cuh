@@ -183,8 +183,21 @@ __device__ __forceinline__ void apply_clover(const void *cl, long stride, long i
         }
 }
 
+#ifndef QX_DSLASH_THREADS
+#define QX_DSLASH_THREADS 128
+#endif
+// Minimum resident CTAs per SM (register cap).  Measured on B200 at 32^3x64
+// (profiles/r01_variants.log): fp32 needs >= 7 x 128 threads in flight per SM to cover HBM
+// latency (72 regs, small L1-resident spills), fp64 must not be capped (152 regs; capping
+// spills and loses 20%).
+template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) ? 1 : 7; };
+#ifdef QX_DSLASH_MINB
+#define QX_MINB_OF(P) QX_DSLASH_MINB
+#else
+#define QX_MINB_OF(P) DslashMinBlocks<P>::value
+#endif
 template <int P, int RECON, bool DAG, int KIND>
-__global__ void __launch_bounds__(128) dslash_kernel(const __grid_constant__ DslashArgs a) {
+__global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
     using R = typename Prec<P>::R;
     const int tid = blockIdx.x * blockDim.x + threadIdx.x;
     if (tid >= a.nthreads) return;
@@ -336,7 +349,7 @@ __global__ void __launch_bounds__(128) dslash_kernel(const __grid_constant__ Dsl
 
 template <int P>
 void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
-    const int threads = 128;
+    const int threads = QX_DSLASH_THREADS;
     const int blocks = (a.nthreads + threads - 1) / threads;
     if (blocks == 0) return;
 #define QX_DS(RC, DG, KD)                                                     \

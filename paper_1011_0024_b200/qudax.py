@@ -15,7 +15,7 @@ import os
 import numpy as np
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "lib", "libqudax.so")
+LIB_PATH = os.environ.get("QUDAX_LIB") or os.path.join(_HERE, "lib", "libqudax.so")  # override: experiments only
 
 HALF, SINGLE, DOUBLE = 2, 4, 8
 EVEN, ODD = 0, 1

@@ -1,0 +1,126 @@
+"""Multi-rank worker (launched by tests/gpu/test_multirank.py through torchrun).
+
+Every rank drives one qudax context on ITS slab of a T-partitioned global lattice.  All ranks
+may share one GPU (the QUDAX_COMM_HOST transport stages faces through pinned host memory and
+exchanges them with torch.distributed/gloo — the paper's non-overlapped strategy),
+or use NCCL when the ranks own distinct GPUs.  Rank 0 gathers the slabs and compares them
+BITWISE with the unpartitioned single-context result (the exchange moves bits only), and the
+solver's solution with the fp64 oracle.
+
+    torchrun --nproc-per-node N tests/gpu/mp_worker.py --comm host|nccl --out result.json
+"""
+import argparse
+import json
+import os
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+sys.path.insert(0, ROOT)
+
+import numpy as np  # noqa: E402
+import torch  # noqa: E402
+import torch.distributed as dist  # noqa: E402
+
+import qgen  # noqa: E402
+from paper_1011_0024_b200 import qudax  # noqa: E402
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--comm", default="host")
+    ap.add_argument("--out", required=True)
+    ap.add_argument("--dims", default="8,4,6,16")
+    ap.add_argument("--same-gpu", type=int, default=1)
+    args = ap.parse_args()
+    dims = tuple(int(v) for v in args.dims.split(","))
+    dist.init_process_group("gloo")
+    rank, n = dist.get_rank(), dist.get_world_size()
+    device = 0 if args.same_gpu else rank
+    torch.cuda.set_device(device)
+    T_loc = dims[3] // n
+    t0 = rank * T_loc
+    U = qgen.gauge(dims, 1301, eps=-1.0, t_begin=t0, nt=T_loc)
+    psi = qgen.spinor(dims, 1302, t_begin=t0, nt=T_loc)
+    xin = qgen.spinor(dims, 1303, t_begin=t0, nt=T_loc)
+    result = {"rank": rank, "n": n, "comm": args.comm, "ok": True, "checks": {}}
+    if args.comm == "nccl":
+        obj = [qudax.nccl_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(obj, src=0)
+        ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_NCCL, nccl_id=obj[0])
+    else:
+        ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_HOST)
+    outs = {}
+    for prec, recon in ((8, 18), (4, 12), (2, 12)):
+        ctx.gauge_load(U, 0.12, 1.0, prec=prec, recon=recon, t_boundary=-1)
+        fi, fo, fx = ctx.new_field(prec), ctx.new_field(prec), ctx.new_field(prec)
+        for p in (0, 1):
+            ctx.spinor_load(fi, prec, 1 - p, psi)
+            ctx.spinor_load(fx, prec, p, xin)
+            for dag in (0, 1):
+                for kind in (0, 1, 2):
+                    ctx.dslash(fo, fi, prec, p, dagger=dag, kind=kind, x=fx, a=-0.3)
+                    outs[(prec, p, dag, kind)] = ctx.spinor_store(fo, prec, p)
+        fa, fb = ctx.new_field(prec), ctx.new_field(prec)
+        ctx.spinor_load(fa, prec, 0, psi)
+        ctx.mdagm(fb, fa, prec)
+        outs[(prec, "mdagm")] = ctx.spinor_store(fb, prec, 0)
+        outs[(prec, "norm2")] = ctx.norm2(fb, prec)
+    # solver across ranks (global reductions through the transport)
+    ctx.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12, t_boundary=-1)
+    b = qgen.point_source(dims, 0, 1, t_begin=t0, nt=T_loc)
+    x, st = ctx.solve(b, tol=1e-10, delta=0.1, maxiter=2000, prec=8, prec_sloppy=4)
+    outs["solve_x"] = x
+    outs["solve_stats"] = st
+    ctx.close()
+
+    # gather slabs to rank 0
+    gathered = [None] * n
+    dist.gather_object(outs, gathered if rank == 0 else None, dst=0)
+    if rank == 0:
+        ref = qudax.Context(dims, device=device)
+        Ug = qgen.gauge(dims, 1301, eps=-1.0)
+        pg, xg = qgen.spinor(dims, 1302), qgen.spinor(dims, 1303)
+        for prec, recon in ((8, 18), (4, 12), (2, 12)):
+            ref.gauge_load(Ug, 0.12, 1.0, prec=prec, recon=recon, t_boundary=-1)
+            fi, fo, fx = ref.new_field(prec), ref.new_field(prec), ref.new_field(prec)
+            for p in (0, 1):
+                ref.spinor_load(fi, prec, 1 - p, pg)
+                ref.spinor_load(fx, prec, p, xg)
+                for dag in (0, 1):
+                    for kind in (0, 1, 2):
+                        ref.dslash(fo, fi, prec, p, dagger=dag, kind=kind, x=fx, a=-0.3)
+                        want = ref.spinor_store(fo, prec, p)
+                        got = np.concatenate([g[(prec, p, dag, kind)] for g in gathered], axis=0)
+                        same = bool(np.array_equal(got, want))
+                        result["checks"][f"dslash p{prec} par{p} dag{dag} kind{kind}"] = same
+                        result["ok"] &= same
+            fa, fb = ref.new_field(prec), ref.new_field(prec)
+            ref.spinor_load(fa, prec, 0, pg)
+            ref.mdagm(fb, fa, prec)
+            got = np.concatenate([g[(prec, "mdagm")] for g in gathered], axis=0)
+            same = bool(np.array_equal(got, ref.spinor_store(fb, prec, 0)))
+            result["checks"][f"mdagm p{prec}"] = same
+            result["ok"] &= same
+            # global norm equals the single-context norm up to summation order
+            n_ref = ref.norm2(fb, prec)
+            close = abs(gathered[0][(prec, "norm2")] - n_ref) <= 1e-12 * n_ref
+            result["checks"][f"norm2 p{prec}"] = close
+            result["ok"] &= close
+        ref.close()
+        # solver: oracle true residual of the gathered solution
+        import oracle
+        wc = oracle.WilsonClover(Ug, 0.124, 1.0, -1.0)
+        xg_ = np.concatenate([g["solve_x"] for g in gathered], axis=0)
+        bg = qgen.point_source(dims, 0, 1)
+        res = float(np.linalg.norm(wc.M(xg_) - bg) / np.linalg.norm(bg))
+        result["solve"] = {"oracle_true_res": res, "stats": gathered[0]["solve_stats"]}
+        okres = res <= 1e-10 * 1.001 and abs(res - gathered[0]["solve_stats"]["true_res"]) <= 1e-9
+        result["checks"]["solve"] = okres
+        result["ok"] &= okres
+        json.dump(result, open(args.out, "w"), indent=1)
+    dist.barrier()
+    dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -1,0 +1,112 @@
+"""Parity at BASELINE.json's full sizes, in the launch configuration bench.py times.
+
+The oracle evaluates the operator only at a sample of output sites (oracle.matpc_sites: the
+same per-site arithmetic as the pinned full-lattice oracle), or — for the solver — the full
+fp64 residual with the clover built chunk by chunk."""
+import numpy as np
+import pytest
+
+import oracle
+import qgen
+from paper_1011_0024_b200 import qudax
+from conftest import TOL
+
+pytestmark = pytest.mark.gpu
+
+KAPPA, CSW = 0.124, 1.0
+
+
+def sample_even_sites(dims, n, seed):
+    X, Y, Z, T = dims
+    rng = np.random.default_rng(seed)
+    lex = rng.choice(X * Y * Z * T, size=4 * n, replace=False)
+    # add sites on the first/last timeslice and the x / y / z edges (ragged boundaries)
+    edge = []
+    for t in (0, T - 1, T // 2):
+        for (x, y, z) in ((0, 0, 0), (X - 1, Y - 1, Z - 1), (X - 1, 0, Z - 1), (1, Y - 1, 0), (0, 1, 1)):
+            edge.append(((t * Z + z) * Y + y) * X + x)
+    lex = np.concatenate([np.array(edge), lex])
+    c = [lex % X, (lex // X) % Y, (lex // (X * Y)) % Z, lex // (X * Y * Z)]
+    even = ((c[0] + c[1] + c[2] + c[3]) % 2) == 0
+    return np.unique(lex[even])[: n + len(edge)]
+
+
+@pytest.fixture(scope="module")
+def config5():
+    dims = (32, 32, 32, 64)  # BASELINE configs[4]: 32^3 x 64 per GPU, the bench workload
+    U = qgen.gauge(dims, 1005, eps=0.1)
+    psi = qgen.spinor(dims, 2005)
+    return dims, U, psi
+
+
+@pytest.mark.parametrize("prec,recon", [(4, 12), (8, 18), (2, 12), (4, 8)])
+def test_matpc_32x64_sampled(torch_cuda, config5, prec, recon):
+    dims, U, psi = config5
+    if recon == 8:
+        U = qgen.gauge(dims, 1005, eps=-1.0)  # 8-reconstruct needs non-degenerate links (reading Q6)
+    ctx = qudax.Context(dims)
+    ctx.gauge_load(U, KAPPA, CSW, prec=prec, recon=recon, t_boundary=-1)
+    fin, fout = ctx.new_field(prec), ctx.new_field(prec)
+    ctx.spinor_load(fin, prec, 0, psi)
+    ctx.matpc(fout, fin, prec)
+    got = ctx.spinor_store(fout, prec, 0).reshape(-1, 4, 3)
+    ctx.close()
+    sites = sample_even_sites(dims, 1500, 11)
+    want = oracle.matpc_sites(U, oracle.restrict(psi, 0), sites, KAPPA, CSW, -1.0)
+    err = np.linalg.norm(got[sites] - want) / np.linalg.norm(want)
+    print(f"32^3x64 prec={prec} recon={recon}: rel-L2 over {len(sites)} sampled sites {err:.2e}")
+    assert err <= TOL[prec]
+
+
+def test_split_path_bitwise_32x64(torch_cuda, config5):
+    """The overlapped interior/boundary split (NCCL loopback) equals the unsplit kernel bitwise
+    at full size."""
+    dims, U, psi = config5
+    outs = []
+    for comm in (qudax.COMM_NONE, qudax.COMM_NCCL):
+        ctx = qudax.Context(dims, comm=comm, nccl_id=qudax.nccl_unique_id() if comm else None)
+        ctx.gauge_load(U, KAPPA, CSW, prec=4, recon=12)
+        fi, fo = ctx.new_field(4), ctx.new_field(4)
+        ctx.spinor_load(fi, 4, 0, psi)
+        ctx.mdagm(fo, fi, 4)
+        ctx.sync()
+        outs.append(fo.cpu().numpy())
+        ctx.close()
+    assert np.array_equal(outs[0], outs[1])
+
+
+def test_strong_scaling_lattice_32x256_sampled(torch_cuda):
+    """BASELINE configs[3] lattice (32^3 x 256) on one GPU: fp32-12 Mhat on sampled sites."""
+    dims = (32, 32, 32, 256)
+    U = qgen.gauge(dims, 1004, eps=0.1)
+    psi = qgen.spinor(dims, 2004)
+    ctx = qudax.Context(dims)
+    ctx.gauge_load(U, KAPPA, CSW, prec=4, recon=12, t_boundary=-1)
+    fin, fout = ctx.new_field(4), ctx.new_field(4)
+    ctx.spinor_load(fin, 4, 0, psi)
+    ctx.matpc(fout, fin, 4)
+    got = ctx.spinor_store(fout, 4, 0).reshape(-1, 4, 3)
+    ctx.close()
+    sites = sample_even_sites(dims, 800, 12)
+    want = oracle.matpc_sites(U, oracle.restrict(psi, 0), sites, KAPPA, CSW, -1.0)
+    assert np.linalg.norm(got[sites] - want) / np.linalg.norm(want) <= TOL[4]
+
+
+def test_config3_mixed_precision_solve(torch_cuda):
+    """BASELINE configs[2]: 24^3 x 128 weak field, fp64 outer + fp32-12 sloppy (delta 0.1) and
+    fp64 outer + half-12 sloppy (delta 1e-2), point source; the oracle's full fp64
+    residual of the solution must meet tol and agree with the reported one to 1e-9."""
+    dims = (24, 24, 24, 128)
+    U = qgen.gauge(dims, 1003, eps=0.1)
+    b = qgen.point_source(dims, 0, 0)
+    ctx = qudax.Context(dims)
+    for ps, delta in ((4, 0.1), (2, 1e-2)):
+        ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=ps, recon_sloppy=12, t_boundary=-1)
+        x, st = ctx.solve(b, tol=1e-12, delta=delta, maxiter=5000, prec=8, prec_sloppy=ps)
+        r = oracle.apply_M_chunked(U, x, KAPPA, CSW, -1.0) - b
+        res = np.linalg.norm(r) / np.linalg.norm(b)
+        print(f"24^3x128 sloppy={ps}: iters {st['iters']} updates {st['reliable_updates']} "
+              f"secs {st['secs']:.3f} reported {st['true_res']:.3e} oracle {res:.3e}")
+        assert res <= 1e-12 * (1 + 1e-3)
+        assert abs(res - st["true_res"]) <= 1e-9
+    ctx.close()

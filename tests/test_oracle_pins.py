@@ -353,3 +353,23 @@ def test_bicgstab_4x4_true_residual():
     assert oracle.true_residual(wc.matpc, xe, bh) < 1e-11
     x = wc.reconstruct(xe, b)
     assert np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b) < 1e-11
+
+
+def test_sampled_evaluation_matches_full():
+    """The site-sampled oracle (used at full BASELINE sizes) is the same per-site arithmetic:
+    it must reproduce the full-lattice D, T and Mhat exactly at the sampled sites."""
+    dims = (4, 4, 2, 6)
+    U = qgen.gauge(dims, 91)
+    psi = qgen.spinor(dims, 92)
+    wc = oracle.WilsonClover(U, 0.12, 1.1, -1.0)
+    rng = np.random.default_rng(3)
+    sites = rng.choice(np.prod(dims), size=20, replace=False)
+    full = oracle.dslash(U, psi, -1.0, True).reshape(-1, 4, 3)
+    assert np.array_equal(oracle.dslash_sites(U, psi, sites, -1.0, True), full[sites])
+    assert np.array_equal(oracle.clover_sites(U, sites, 0.12, 1.1), wc.T.reshape(-1, 12, 12)[sites])
+    odd = oracle.parity_mask(dims).reshape(-1)
+    ev = np.nonzero(~odd)[0][::3]
+    psi_e = oracle.restrict(psi, 0)
+    got = oracle.matpc_sites(U, psi_e, ev, 0.12, 1.1, -1.0)
+    want = wc.matpc(psi_e).reshape(-1, 4, 3)[ev]
+    assert np.abs(got - want).max() < 1e-13
