@@ -113,35 +113,62 @@ struct Blocks<4, NB, STREAM> {
     }
 };
 
+// ---- 16-bit fixed point <-> fp32 without the conversion (XU) pipe ------------------------
+// The paper's half precision relied on the GT200 texture unit to turn int16 into floats
+// (P:509-518).  On B200, I2F/F2I issue on the narrow XU pipe and become the limiter of the
+// half-precision Dslash (ncu: XU 60% busy).  Both directions are done with exact fp32
+// integer tricks on the ALU/FMA pipes instead:
+//   int16 s -> float: bits(0x4B000000 | (u16(s) ^ 0x8000)) = 2^23 + s + 2^15 exactly, minus
+//   (2^23 + 2^15);  float x (|x| <= 32767) -> RN-even int16: low 16 bits of bits(x + 1.5*2^23).
+__device__ __forceinline__ float i16lo_to_f32(uint32_t w) {
+    return __uint_as_float((w & 0xFFFFu) ^ 0x4B008000u) - 8421376.0f;
+}
+__device__ __forceinline__ float i16hi_to_f32(uint32_t w) {
+    return __uint_as_float((w >> 16) ^ 0x4B008000u) - 8421376.0f;
+}
+// two already-scaled floats -> packed int16 pair (round to nearest even, as __float2int_rn)
+__device__ __forceinline__ uint32_t f32x2_to_i16x2(float a, float b) {
+    const uint32_t ia = __float_as_uint(__fadd_rn(a, 12582912.0f));
+    const uint32_t ib = __float_as_uint(__fadd_rn(b, 12582912.0f));
+    return __byte_perm(ia, ib, 0x5410);
+}
+// the integer value held in a quantised word, as a float (exact)
+__device__ __forceinline__ float q_as_f32(float scaled) {
+    return __uint_as_float(__float_as_uint(__fadd_rn(scaled, 12582912.0f))) - 12582912.0f;
+}
+__device__ __forceinline__ uint2 ld_stream_u2(const uint2 *p) {
+    uint2 v;
+    asm volatile("ld.global.nc.L1::no_allocate.v2.u32 {%0,%1}, [%2];" : "=r"(v.x), "=r"(v.y) : "l"(p));
+    return v;
+}
+
 // half: raw integer values scaled by `scale` (norm/32767 for spinors, 1/32767 for links)
 template <int NB, bool STREAM>
 struct Blocks<2, NB, STREAM> {
     static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out,
                                                 float scale) {
-        const short4 *p = reinterpret_cast<const short4 *>(base);
+        const uint2 *p = reinterpret_cast<const uint2 *>(base);
 #pragma unroll
         for (int k = 0; k < NB; ++k) {
-            short4 v = STREAM ? ld_stream(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
-            out[4 * k] = scale * (float)v.x;
-            out[4 * k + 1] = scale * (float)v.y;
-            out[4 * k + 2] = scale * (float)v.z;
-            out[4 * k + 3] = scale * (float)v.w;
+            uint2 v = STREAM ? ld_stream_u2(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
+            out[4 * k] = __fmul_rn(scale, i16lo_to_f32(v.x));
+            out[4 * k + 1] = __fmul_rn(scale, i16hi_to_f32(v.x));
+            out[4 * k + 2] = __fmul_rn(scale, i16lo_to_f32(v.y));
+            out[4 * k + 3] = __fmul_rn(scale, i16hi_to_f32(v.y));
         }
     }
     static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out) {
         load(base, stride, i, b0, out, kHalfInv);
     }
-    // store already-quantised values
+    // quantise (value * inv_scale, round to nearest even) and store
     static __device__ __forceinline__ void store_q(void *base, long stride, long i, int b0, const float *in,
                                                    float inv_scale) {
-        short4 *p = reinterpret_cast<short4 *>(base);
+        uint2 *p = reinterpret_cast<uint2 *>(base);
 #pragma unroll
         for (int k = 0; k < NB; ++k) {
-            short4 v;
-            v.x = (short)__float2int_rn(in[4 * k] * inv_scale);
-            v.y = (short)__float2int_rn(in[4 * k + 1] * inv_scale);
-            v.z = (short)__float2int_rn(in[4 * k + 2] * inv_scale);
-            v.w = (short)__float2int_rn(in[4 * k + 3] * inv_scale);
+            uint2 v;
+            v.x = f32x2_to_i16x2(__fmul_rn(in[4 * k], inv_scale), __fmul_rn(in[4 * k + 1], inv_scale));
+            v.y = f32x2_to_i16x2(__fmul_rn(in[4 * k + 2], inv_scale), __fmul_rn(in[4 * k + 3], inv_scale));
             p[(b0 + k) * stride + i] = v;
         }
     }
@@ -200,7 +227,7 @@ struct SpinorIO {
             const float inv = (m > 0.f) ? kHalfMax / m : 0.f;
             const float scale = m * kHalfInv;
 #pragma unroll
-            for (int k = 0; k < 24; ++k) v[k] = scale * (float)(short)__float2int_rn(v[k] * inv);
+            for (int k = 0; k < 24; ++k) v[k] = __fmul_rn(scale, q_as_f32(__fmul_rn(v[k], inv)));
         }
     }
 };
@@ -247,9 +274,9 @@ struct LinkIO {
             } else {
                 const short2 *p2 = reinterpret_cast<const short2 *>(reinterpret_cast<const char *>(base) +
                                                                     (size_t)NB4 * 8 * stride);
-                short2 v = ld_stream(p2 + i);
-                raw[RECON - 2] = kHalfInv * (float)v.x;
-                raw[RECON - 1] = kHalfInv * (float)v.y;
+                const uint32_t w = __ldg(reinterpret_cast<const uint32_t *>(p2) + i);
+                raw[RECON - 2] = __fmul_rn(kHalfInv, i16lo_to_f32(w));
+                raw[RECON - 1] = __fmul_rn(kHalfInv, i16hi_to_f32(w));
             }
         }
     }
@@ -280,14 +307,14 @@ struct LinkIO {
             }
             Cx<R> u01 = cx(raw[2], raw[3]), u02 = cx(raw[4], raw[5]), u10 = cx(raw[6], raw[7]);
             R n = norm2(u01) + norm2(u02);
-            R a00 = sqrt(fmax((R)0, (R)1 - n));
+            R a00 = sqrt_(fmax((R)0, (R)1 - n));
             R s0, c0, s2, c2;
             sincos_(th0, &s0, &c0);
             sincos_(th2, &s2, &c2);
             Cx<R> u00 = cx(a00 * c0, a00 * s0);
-            R a20 = sqrt(fmax((R)0, (R)1 - a00 * a00 - norm2(u10)));
+            R a20 = sqrt_(fmax((R)0, (R)1 - a00 * a00 - norm2(u10)));
             Cx<R> u20 = cx(a20 * c2, a20 * s2);
-            R inv = (R)1 / n;
+            R inv = rcp_(n);
             Cx<R> A = conj_mul(u00, u10);
             Cx<R> C = conj_mul(u00, u20);
             Cx<R> cu20 = conj(u20), cu10 = conj(u10), cu01 = conj(u01), cu02 = conj(u02);
@@ -301,8 +328,14 @@ struct LinkIO {
         }
     }
 
+    // fp64: accurate; fp32/half: SFU approximations (abs error ~4e-7 on [-pi, pi], far inside
+    // the 1e-5 / 5e-3 budgets) — the accurate fp32 versions made recon-8 instruction-bound
     static __device__ __forceinline__ void sincos_(double x, double *s, double *c) { sincos(x, s, c); }
-    static __device__ __forceinline__ void sincos_(float x, float *s, float *c) { sincosf(x, s, c); }
+    static __device__ __forceinline__ void sincos_(float x, float *s, float *c) { __sincosf(x, s, c); }
+    static __device__ __forceinline__ double sqrt_(double x) { return sqrt(x); }
+    static __device__ __forceinline__ float sqrt_(float x) { return x * rsqrtf(fmaxf(x, 1e-30f)); }
+    static __device__ __forceinline__ double rcp_(double x) { return 1.0 / x; }
+    static __device__ __forceinline__ float rcp_(float x) { return __fdividef(1.0f, x); }
 };
 
 }  // namespace qx

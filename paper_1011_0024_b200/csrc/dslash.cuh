@@ -220,10 +220,27 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     const int lex = ((t * Z + z) * Y + y) * X + x;
 
     Cx<R> acc[4][3];
+    // xpay: out = T x + a D in.  The site-local T x is computed FIRST and carried in the
+    // accumulator as (1/a) T x, so its loads (x, clover) overlap the stencil's instead of
+    // adding a dependent memory round trip after it; out = a * acc at the end.
+    const bool xpay_early = (KIND == QUDAX_CLOVER_XPAY) && (a.a != 0.0);
+    if (xpay_early) {
+        R v[24];
+        Cx<R> xs[4][3];
+        SpinorIO<P>::load(a.x, a.stride, i, v);
+        unpack_spinor(v, xs);
+        apply_clover<P>(a.clover, a.stride, i, xs, acc);
+        const R inv_a = (R)(1.0 / a.a);
 #pragma unroll
-    for (int s = 0; s < 4; ++s)
+        for (int s = 0; s < 4; ++s)
 #pragma unroll
-        for (int c = 0; c < 3; ++c) acc[s][c] = cx((R)0, (R)0);
+            for (int c = 0; c < 3; ++c) acc[s][c] = inv_a * acc[s][c];
+    } else {
+#pragma unroll
+        for (int s = 0; s < 4; ++s)
+#pragma unroll
+            for (int c = 0; c < 3; ++c) acc[s][c] = cx((R)0, (R)0);
+    }
 
     constexpr int SF = DAG ? +1 : -1;  // sigma of the forward hop
     constexpr int SB = -SF;
@@ -324,17 +341,18 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
             for (int c = 0; c < 3; ++c) res[s][c] = acc[s][c];
     } else if constexpr (KIND == QUDAX_CLOVER_INV) {
         apply_clover<P>(a.clover, a.stride, i, acc, res);
-    } else {
+    } else if (xpay_early) {
+        const R co = (R)a.a;
+#pragma unroll
+        for (int s = 0; s < 4; ++s)
+#pragma unroll
+            for (int c = 0; c < 3; ++c) res[s][c] = co * acc[s][c];
+    } else {  // a == 0: out = T x
         R v[24];
         Cx<R> xs[4][3];
         SpinorIO<P>::load(a.x, a.stride, i, v);
         unpack_spinor(v, xs);
         apply_clover<P>(a.clover, a.stride, i, xs, res);
-        const R co = (R)a.a;
-#pragma unroll
-        for (int s = 0; s < 4; ++s)
-#pragma unroll
-            for (int c = 0; c < 3; ++c) res[s][c] = res[s][c] + co * acc[s][c];
     }
     R o[24];
 #pragma unroll
