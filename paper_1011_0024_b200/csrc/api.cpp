@@ -8,6 +8,7 @@
 #include <algorithm>
 #include <chrono>
 #include <cmath>
+#include <cstdlib>
 #include <cstring>
 
 #include "ctx.h"
@@ -113,6 +114,8 @@ static void exchange(qudax_ctx *c, const void *send_fwd, const void *send_back, 
     }
 }
 
+static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res);
+
 static cudaEvent_t pool_event(qudax_ctx *c) {
     if (!c->ev_pool.empty()) {
         cudaEvent_t e = c->ev_pool.back();
@@ -122,6 +125,12 @@ static cudaEvent_t pool_event(qudax_ctx *c) {
     cudaEvent_t e;
     QX_CUDA(cudaEventCreate(&e));
     return e;
+}
+
+static int dslash_blocks_any(int prec, int recon, int dagger, int kind, int nthreads) {
+    if (prec == 8) return dslash_blocks_f64(recon, dagger, kind, nthreads);
+    if (prec == 4) return dslash_blocks_f32(recon, dagger, kind, nthreads);
+    return dslash_blocks_f16(recon, dagger, kind, nthreads);
 }
 
 static void launch_dslash_raw(int prec, int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
@@ -139,14 +148,45 @@ static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int
         return;
     }
     qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads};
+    if (c->capturing) {  // graph: external event-record nodes, re-recorded at each replay
+        QX_CUDA(cudaEventRecordWithFlags(r.a, c->stream, cudaEventRecordExternal));
+        launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
+        QX_CUDA(cudaEventRecordWithFlags(r.b, c->stream, cudaEventRecordExternal));
+        c->graph_trecs.push_back(r);
+        return;
+    }
     QX_CUDA(cudaEventRecord(r.a, c->stream));
     launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
     QX_CUDA(cudaEventRecord(r.b, c->stream));
     c->trecs.push_back(r);
 }
 
+void harvest_graph_timing(qudax_ctx *c) {
+    for (auto &r : c->graph_trecs) {
+        float ms = 0;
+        QX_CUDA(cudaEventElapsedTime(&ms, r.a, r.b));
+        qudax_site_model m;
+        qudax_model(r.prec, r.recon, r.kind, &m);
+        auto &t = c->tacc[prec_idx(r.prec)];
+        t.launches += 1;
+        t.sites += r.sites;
+        t.ms += ms;
+        t.flops += m.flops * r.sites;
+        t.bytes_c += m.bytes_compulsory * r.sites;
+        t.bytes_p += m.bytes_paper * r.sites;
+    }
+}
+
+void release_graph_timing(qudax_ctx *c) {
+    for (auto &r : c->graph_trecs) {
+        c->ev_pool.push_back(r.a);
+        c->ev_pool.push_back(r.b);
+    }
+    c->graph_trecs.clear();
+}
+
 void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
-               double a) {
+               double a, const RedReq *red, int reverse) {
     check_prec(prec);
     QX_CHECK(p == 0 || p == 1, QUDAX_ERR_ARG, "parity must be 0 or 1");
     QX_CHECK(kind >= 0 && kind <= 2, QUDAX_ERR_ARG, "bad dslash kind");
@@ -162,6 +202,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     args.bc_fwd = (g.rank == g.nranks - 1) ? (double)c->t_bc : 1.0;
     args.bc_back = (g.rank == 0) ? (double)c->t_bc : 1.0;
     args.a = a;
+    args.reverse = reverse;
     args.in = in; args.out = out; args.x = x;
     for (int m = 0; m < 4; ++m)
         for (int q = 0; q < 2; ++q) args.gauge[m][q] = gc.d[m][q];
@@ -171,12 +212,44 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         QX_CHECK(cl.valid, QUDAX_ERR_STATE, "no clover in this precision");
         args.clover = (kind == QUDAX_CLOVER_XPAY) ? cl.T[p] : cl.Tinv[p];
     }
+    int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
+    const int TPB = dslash_threads();
+    const bool split = (c->comm == QUDAX_COMM_NCCL && c->overlap && g.T_loc > 2);
+    const bool multi = (g.nranks > 1);  // cross-rank sums needed before the scalar recurrence
+    if (red) {
+        QX_CHECK(red->kind != RED_XDOT_NORM || kind == QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
+        QX_CHECK(red->kind != RED_RHAT_DOT || red->rhat, QUDAX_ERR_ARG, "rhat-dot needs rhat");
+        // CTA slots of up to two launches + their group slots (reduce.cuh)
+        if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / TPB) + 64)));
+        args.red_kind = red->kind;
+        args.rhat = red->rhat;
+        const int ni = (int)((g.T_loc - 2) * g.F), nb = (int)(2 * g.F);
+        args.tail.partials = c->dpart;
+        args.tail.counter = c->d_counter;
+        args.tail.total_blocks = split ? dslash_blocks_any(prec, gc.recon, dagger, kind, ni) +
+                                             dslash_blocks_any(prec, gc.recon, dagger, kind, nb)
+                                       : dslash_blocks_any(prec, gc.recon, dagger, kind, (int)g.Vh);
+        args.tail.out = red->S ? red->S->red : c->red_out;
+        args.tail.S = red->S;
+        args.tail.coef_mode = (red->S && !multi) ? red->coef_mode : COEF_NONE;
+    }
+    auto launch = [&](int range, int nthreads) {
+        args.range = range;
+        args.nthreads = nthreads;
+        args.tail.block_offset = red_blocks;
+        launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
+        red_blocks += dslash_blocks_any(prec, gc.recon, dagger, kind, nthreads);
+        c->launches += 1;
+    };
+    auto finish_red = [&] {
+        if (!red) return;
+        if (!red->S) global_sum(c, c->red_out, 3, red->res);
+        else if (multi) device_sum_coef(c, red->S->red, 3, red->S, red->coef_mode);
+    };
     if (c->comm == QUDAX_COMM_NONE) {
         args.ghosted = 0;
-        args.range = RANGE_ALL;
-        args.nthreads = (int)g.Vh;
-        launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
-        c->launches += 1;
+        launch(RANGE_ALL, (int)g.Vh);
+        finish_red();
         return;
     }
     auto &h = halo_for(c, prec);
@@ -191,30 +264,21 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         exchange(c, h.sf, h.sb, h.gb, h.gf, h.bytes, c->comm_stream, nullptr, nullptr, nullptr, nullptr);
         QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
         c->launches += 1;
-        if (c->overlap && g.T_loc > 2) {
-            args.range = RANGE_INTERIOR;
-            args.nthreads = (int)((g.T_loc - 2) * g.F);
-            launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
+        if (split) {
+            launch(RANGE_INTERIOR, (int)((g.T_loc - 2) * g.F));
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
-            args.range = RANGE_BOUNDARY;
-            args.nthreads = (int)(2 * g.F);
-            launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
-            c->launches += 2;
+            launch(RANGE_BOUNDARY, (int)(2 * g.F));
         } else {
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
-            args.range = RANGE_ALL;
-            args.nthreads = (int)g.Vh;
-            launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
-            c->launches += 1;
+            launch(RANGE_ALL, (int)g.Vh);
         }
     } else {  // HOST: paper strategy 1 (no overlap)
         launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, c->stream);
         exchange(c, h.sf, h.sb, h.gb, h.gf, h.bytes, c->stream, h.h_sf, h.h_sb, h.h_gb, h.h_gf);
-        args.range = RANGE_ALL;
-        args.nthreads = (int)g.Vh;
-        launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
-        c->launches += 2;
+        c->launches += 1;
+        launch(RANGE_ALL, (int)g.Vh);
     }
+    finish_red();
 }
 
 static void *tmp_odd(qudax_ctx *c, int prec) {
@@ -229,10 +293,12 @@ static void *tmp_even(qudax_ctx *c, int prec) {
 }
 
 // Mhat = T_ee - kappa^2 D_eo T_oo^{-1} D_oe (asymmetric Schur form on even sites)
-void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger) {
+void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red) {
     void *t = tmp_odd(c, prec);
-    dslash_op(c, t, in, nullptr, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0);
-    dslash_op(c, out, t, in, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa);
+    dslash_op(c, t, in, nullptr, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, nullptr);
+    // the second kernel walks the lattice top-down: the timeslices the first kernel touched
+    // last (their links, T^{-1} D in and the dirty tmp lines) are still in the 126 MB L2
+    dslash_op(c, out, t, in, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, red, 1);
 }
 
 void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int parity, bool inverse) {
@@ -255,10 +321,43 @@ static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res) {
 }
 
 int blas_op(qudax_ctx *c, int op, int prec, void *const *f, const double *coef, double *res) {
-    int n = blas_run(op, prec, c->g, f, coef, c->partials, c->red_out, c->stream);
-    c->launches += 1 + (n ? 1 : 0);
+    CoefArg co[2] = {};
+    if (coef) {
+        co[0].v = make_double2(coef[0], op == OP_XPAY ? 0.0 : coef[1]);
+        if (op == OP_P_UPDATE || op == OP_FINAL) co[1].v = make_double2(coef[2], coef[3]);
+    }
+    RedTail tail{c->partials, c->d_counter, 0, 0, c->red_out, nullptr, COEF_NONE};
+    int n = blas_run(op, prec, c->g, f, co, tail, c->stream);
+    c->launches += 1;
     if (n) global_sum(c, c->red_out, n, res);
     return n;
+}
+
+// Global sum of n device doubles in place (stream-ordered, no host round trip for NCCL / one
+// rank), then the device-side scalar recurrence `mode` (launch_coef).
+void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, int mode) {
+    if (c->g.nranks > 1 && c->comm == QUDAX_COMM_NCCL) {
+        QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl, c->stream));
+    } else if (c->g.nranks > 1 && c->comm == QUDAX_COMM_HOST) {
+        QX_CUDA(cudaMemcpyAsync(c->h_red, dev_vals, sizeof(double) * n, cudaMemcpyDeviceToHost, c->stream));
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        if (c->host_allreduce(c->h_red, n, c->comm_user)) throw Error(QUDAX_ERR_COMM, "host_allreduce hook failed");
+        QX_CUDA(cudaMemcpyAsync(dev_vals, c->h_red, sizeof(double) * n, cudaMemcpyHostToDevice, c->stream));
+    }
+    if (mode != COEF_NONE) {
+        launch_coef(S, mode, c->stream);
+        c->launches += 1;
+    }
+}
+
+// BLAS op whose coefficients may live on the device; its reduction (if any) goes to S->red,
+// is summed over ranks and fed to the scalar recurrence `mode` — all stream-ordered.
+void blas_op_dev(qudax_ctx *c, int op, int prec, void *const *f, const CoefArg *co, SolverScalars *S, int mode) {
+    const bool multi = c->g.nranks > 1;
+    RedTail tail{c->partials, c->d_counter, 0, 0, S->red, S, multi ? COEF_NONE : mode};
+    int n = blas_run(op, prec, c->g, f, co, tail, c->stream);
+    c->launches += 1;
+    if (n && multi) device_sum_coef(c, S->red, n, S, mode);
 }
 
 void xpy_mixed_op(qudax_ctx *c, int pd, int ps, const void *x, void *y) {
@@ -506,6 +605,7 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         g.fstride = pad64(g.F);
         QX_CHECK(g.V < (1L << 30), QUDAX_ERR_ARG, "local volume too large for 32-bit site indexing");
         c->device = p->device;
+        if (const char *ng = std::getenv("QUDAX_NO_GRAPHS")) c->no_graphs = (ng[0] == '1');
         c->comm = p->comm;
         c->overlap = p->overlap;
         c->dev_alloc = p->dev_alloc; c->dev_free = p->dev_free; c->alloc_user = p->alloc_user;
@@ -531,6 +631,10 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         c->red_out = static_cast<double *>(dalloc(c, sizeof(double) * 8));
         c->h_red = static_cast<double *>(halloc(c, sizeof(double) * 8));
         c->d_flag = static_cast<int *>(dalloc(c, sizeof(int) * 4));
+        // reduction tail counters: [0] groups done, [1 + g] CTAs done in group g (reduce.cuh)
+        const size_t ncount = 2 + (size_t)(g.Vh / 32) / 64 + 64;
+        c->d_counter = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * ncount));
+        QX_CUDA(cudaMemsetAsync(c->d_counter, 0, sizeof(unsigned) * ncount, c->stream));
     });
     if (st != QUDAX_OK) {
         qudax_finalize(c);
@@ -551,6 +655,7 @@ qudax_status qudax_finalize(qudax_ctx *c) {
     }
     for (void *p : c->host_allocs) cudaFreeHost(p);
     for (auto &r : c->trecs) { cudaEventDestroy(r.a); cudaEventDestroy(r.b); }
+    for (auto &r : c->graph_trecs) { cudaEventDestroy(r.a); cudaEventDestroy(r.b); }
     for (auto e : c->ev_pool) cudaEventDestroy(e);
     if (c->ev_in) cudaEventDestroy(c->ev_in);
     if (c->ev_halo) cudaEventDestroy(c->ev_halo);
@@ -587,6 +692,7 @@ qudax_status qudax_kernel_timing(qudax_ctx *c, int enable) {
             c->ev_pool.push_back(r.b);
         }
         c->trecs.clear();
+        for (auto &t : c->tacc) t = qudax_ctx::TimingAcc{};
         c->timing = enable != 0;
     });
 }
@@ -608,6 +714,17 @@ qudax_status qudax_get_kernel_stats(qudax_ctx *c, int prec_filter, qudax_kernel_
             o->flops += m.flops * r.sites;
             o->bytes_compulsory += m.bytes_compulsory * r.sites;
             o->bytes_paper += m.bytes_paper * r.sites;
+        }
+        for (int q = 0; q < 3; ++q) {
+            const int pr = q == 0 ? 8 : (q == 1 ? 4 : 2);
+            if (prec_filter && pr != prec_filter) continue;
+            const auto &t = c->tacc[q];
+            o->launches += t.launches;
+            o->sites += t.sites;
+            o->ms_total += t.ms;
+            o->flops += t.flops;
+            o->bytes_compulsory += t.bytes_c;
+            o->bytes_paper += t.bytes_p;
         }
     });
 }

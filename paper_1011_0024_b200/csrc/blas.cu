@@ -2,67 +2,65 @@
 // fusion wherever possible to reduce memory traffic"; P:721-725 global sums).  All vectors
 // are parity fields (V_h sites) in the site-major SoA of one precision; arithmetic is in the
 // storage precision's compute type (fp32 for half), every reduction accumulates in fp64 and
-// is reduced deterministically: per-CTA partials in a fixed grid, then one CTA sums them in
-// a fixed order (reading Q12), so results are bitwise reproducible run to run.
+// is reduced deterministically (reduce.cuh: fixed per-CTA slots, the last CTA sums them in a
+// fixed order — reading Q12), so results are bitwise reproducible run to run.
+// Coefficients are either values or device scalars (CoefArg), so the solver iteration can run
+// without host round trips.
+#include <mutex>
+#include <unordered_map>
+
 #include "core.cuh"
-#include "dslash.cuh"
 #include "internal.h"
+#include "reduce.cuh"
 
 namespace qx {
 
 constexpr int kBlasThreads = 256;
-constexpr int kBlasBlocks = 148 * 4;  // fixed grid: 4 CTAs per SM on 148 SMs
+constexpr int kBlasMaxBlocks = 160 * 8;  // partials capacity: <= 8 resident 256-thread CTAs per SM
 
-int blas_partial_blocks() { return kBlasBlocks; }
+int blas_partial_blocks() { return kBlasMaxBlocks; }
+
+// Exactly one full wave: SMs x resident CTAs per SM for this kernel (a fixed multiple of 148
+// that does not fit one wave leaves a ragged second wave).  Cached per kernel; the grid is a
+// property of the kernel and the device only, so the reductions stay deterministic.
+template <typename K>
+static int one_wave(K kernel) {
+    static std::mutex mu;
+    static std::unordered_map<const void *, int> cache;
+    std::lock_guard<std::mutex> lk(mu);
+    auto it = cache.find((const void *)kernel);
+    if (it != cache.end()) return it->second;
+    int dev = 0, sms = 0, per = 0;
+    QX_CUDA(cudaGetDevice(&dev));
+    QX_CUDA(cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev));
+    QX_CUDA(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per, kernel, kBlasThreads, 0));
+    int b = sms * (per > 0 ? per : 1);
+    if (b > kBlasMaxBlocks) b = kBlasMaxBlocks;
+    cache[(const void *)kernel] = b;
+    return b;
+}
 
 template <int NRED>
-__device__ __forceinline__ void block_reduce_store(double (&v)[NRED], double *partials) {
-    __shared__ double sm[kBlasThreads / 32][NRED > 0 ? NRED : 1];
-#pragma unroll
-    for (int k = 0; k < NRED; ++k)
-#pragma unroll
-        for (int o = 16; o > 0; o >>= 1) v[k] += __shfl_xor_sync(0xffffffffu, v[k], o);
-    const int w = threadIdx.x / 32, l = threadIdx.x % 32;
-    if (l == 0)
-#pragma unroll
-        for (int k = 0; k < NRED; ++k) sm[w][k] = v[k];
-    __syncthreads();
-    if (threadIdx.x < NRED) {
-        double s = 0;
-        for (int ww = 0; ww < kBlasThreads / 32; ++ww) s += sm[ww][threadIdx.x];
-        partials[blockIdx.x * NRED + threadIdx.x] = s;
-    }
+__device__ __forceinline__ void block_reduce_store(double (&v)[NRED], const RedTail &t) {
+    reduce_with_tail<NRED, kBlasThreads>(v, t);
 }
 
-// single CTA: out[k] = sum_b partials[b * nred + k], fixed order
-__global__ void k_reduce_final(const double *__restrict__ partials, int nblocks, int nred, double *out) {
-    __shared__ double sm[kBlasThreads];
-    for (int k = 0; k < nred; ++k) {
-        double s = 0;
-        for (int b = threadIdx.x; b < nblocks; b += blockDim.x) s += partials[b * nred + k];
-        sm[threadIdx.x] = s;
-        __syncthreads();
-        for (int w = blockDim.x / 2; w > 0; w >>= 1) {
-            if (threadIdx.x < w) sm[threadIdx.x] += sm[threadIdx.x + w];
-            __syncthreads();
-        }
-        if (threadIdx.x == 0) out[k] = sm[0];
-        __syncthreads();
-    }
+// BiCGstab scalar recurrence after a multi-rank allreduce of S->red (single thread)
+__global__ void k_coef(SolverScalars *S, int mode) { apply_coef(S, mode); }
+void launch_coef(SolverScalars *S, int mode, cudaStream_t s) {
+    k_coef<<<1, 1, 0, s>>>(S, mode);
+    QX_CUDA(cudaGetLastError());
 }
 
-template <typename R>
-using Sp = R[24];
-
-// ---------------------------------------------------------------------------- kernels
-// y = x + c * y ... each kernel documents its formula; c* are complex (re, im) as double2.
+#define QX_GRID_LOOP(i) for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x)
 
 // p <- r + beta (p - omega v)            (BiCGstab search direction)
 template <int P>
-__global__ void k_p_update(long Vh, long stride, const void *r, void *p, const void *v, double2 beta, double2 omega) {
+__global__ void k_p_update(long Vh, long stride, const void *r, void *p, const void *v, CoefArg beta_, CoefArg omega_) {
     using R = typename Prec<P>::R;
+    const double2 beta = coef_get(beta_), omega = coef_get(omega_);
     const Cx<R> b = cx((R)beta.x, (R)beta.y), w = cx((R)omega.x, (R)omega.y);
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         R rr[24], pp[24], vv[24];
         SpinorIO<P>::load(r, stride, i, rr);
         SpinorIO<P>::load(p, stride, i, pp);
@@ -80,10 +78,11 @@ __global__ void k_p_update(long Vh, long stride, const void *r, void *p, const v
 
 // y <- y + c x   (c complex)
 template <int P>
-__global__ void k_caxpy(long Vh, long stride, double2 c, const void *x, void *y) {
+__global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y) {
     using R = typename Prec<P>::R;
+    const double2 c = coef_get(c_);
     const Cx<R> a = cx((R)c.x, (R)c.y);
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         R xx[24], yy[24];
         SpinorIO<P>::load(x, stride, i, xx);
         SpinorIO<P>::load(y, stride, i, yy);
@@ -101,7 +100,7 @@ __global__ void k_caxpy(long Vh, long stride, double2 c, const void *x, void *y)
 template <int P>
 __global__ void k_xpay(long Vh, long stride, const void *x, double a, const void *y, void *z) {
     using R = typename Prec<P>::R;
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         R xx[24], yy[24];
         SpinorIO<P>::load(x, stride, i, xx);
         SpinorIO<P>::load(y, stride, i, yy);
@@ -113,10 +112,10 @@ __global__ void k_xpay(long Vh, long stride, const void *x, double a, const void
 
 // sum conj(a) b -> (re, im)
 template <int P>
-__global__ void k_cdot(long Vh, long stride, const void *a, const void *b, double *partials) {
+__global__ void k_cdot(long Vh, long stride, const void *a, const void *b, RedTail tail) {
     using R = typename Prec<P>::R;
     double acc[2] = {0, 0};
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         R aa[24], bb[24];
         SpinorIO<P>::load(a, stride, i, aa);
         SpinorIO<P>::load(b, stride, i, bb);
@@ -126,29 +125,29 @@ __global__ void k_cdot(long Vh, long stride, const void *a, const void *b, doubl
             acc[1] += (double)aa[2 * k] * bb[2 * k + 1] - (double)aa[2 * k + 1] * bb[2 * k];
         }
     }
-    block_reduce_store<2>(acc, partials);
+    block_reduce_store<2>(acc, tail);
 }
 
 // sum |a|^2
 template <int P>
-__global__ void k_norm2(long Vh, long stride, const void *a, double *partials) {
+__global__ void k_norm2(long Vh, long stride, const void *a, RedTail tail) {
     using R = typename Prec<P>::R;
     double acc[1] = {0};
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         R aa[24];
         SpinorIO<P>::load(a, stride, i, aa);
 #pragma unroll
         for (int k = 0; k < 24; ++k) acc[0] += (double)aa[k] * aa[k];
     }
-    block_reduce_store<1>(acc, partials);
+    block_reduce_store<1>(acc, tail);
 }
 
 // (<t, s>, |t|^2)
 template <int P>
-__global__ void k_tdot(long Vh, long stride, const void *t, const void *s, double *partials) {
+__global__ void k_tdot(long Vh, long stride, const void *t, const void *s, RedTail tail) {
     using R = typename Prec<P>::R;
     double acc[3] = {0, 0, 0};
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         R tt[24], ss[24];
         SpinorIO<P>::load(t, stride, i, tt);
         SpinorIO<P>::load(s, stride, i, ss);
@@ -159,17 +158,18 @@ __global__ void k_tdot(long Vh, long stride, const void *t, const void *s, doubl
             acc[2] += (double)tt[2 * k] * tt[2 * k] + (double)tt[2 * k + 1] * tt[2 * k + 1];
         }
     }
-    block_reduce_store<3>(acc, partials);
+    block_reduce_store<3>(acc, tail);
 }
 
 // x <- x + alpha p + omega s ; s <- s - omega t ; returns (|s|^2, <rhat, s>) of the new s
 template <int P>
 __global__ void k_bicg_final(long Vh, long stride, void *x, const void *p, void *s, const void *t, const void *rhat,
-                             double2 alpha, double2 omega, double *partials) {
+                             CoefArg alpha_, CoefArg omega_, RedTail tail) {
     using R = typename Prec<P>::R;
+    const double2 alpha = coef_get(alpha_), omega = coef_get(omega_);
     const Cx<R> al = cx((R)alpha.x, (R)alpha.y), om = cx((R)omega.x, (R)omega.y);
     double acc[3] = {0, 0, 0};
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         R xx[24], pp[24], ss[24];
         SpinorIO<P>::load(x, stride, i, xx);
         SpinorIO<P>::load(p, stride, i, pp);
@@ -199,13 +199,13 @@ __global__ void k_bicg_final(long Vh, long stride, void *x, const void *p, void 
             acc[2] += (double)rh[2 * k] * ss[2 * k + 1] - (double)rh[2 * k + 1] * ss[2 * k];
         }
     }
-    block_reduce_store<3>(acc, partials);
+    block_reduce_store<3>(acc, tail);
 }
 
 // y(PD) <- y(PD) + x(PS)
 template <int PD, int PS>
 __global__ void k_xpy_mixed(long Vh, long stride, const void *x, void *y) {
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         typename Prec<PS>::R xx[24];
         typename Prec<PD>::R yy[24];
         SpinorIO<PS>::load(x, stride, i, xx);
@@ -218,10 +218,10 @@ __global__ void k_xpy_mixed(long Vh, long stride, const void *x, void *y) {
 
 // r <- b - r ; returns |r|^2
 template <int P>
-__global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, double *partials) {
+__global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, RedTail tail) {
     using R = typename Prec<P>::R;
     double acc[1] = {0};
-    for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x) {
+    QX_GRID_LOOP(i) {
         R bb[24], rr[24];
         SpinorIO<P>::load(b, stride, i, bb);
         SpinorIO<P>::load(r, stride, i, rr);
@@ -231,7 +231,7 @@ __global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, double 
 #pragma unroll
         for (int k = 0; k < 24; ++k) acc[0] += (double)rr[k] * rr[k];
     }
-    block_reduce_store<1>(acc, partials);
+    block_reduce_store<1>(acc, tail);
 }
 
 // ---------------------------------------------------------------------------- dispatch
@@ -243,60 +243,59 @@ __global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, double 
         default: throw Error(QUDAX_ERR_ARG, "blas: bad precision"); \
     }
 
-static inline double2 d2(const double *c) { return make_double2(c[0], c[1]); }
+// one launch of kernel K on its one-wave grid; for reducing kernels the tail spans that grid
+#define QX_LAUNCH(K, ...)                              \
+    do {                                               \
+        const int B_ = one_wave(K);                    \
+        tail.total_blocks = B_;                        \
+        tail.block_offset = 0;                         \
+        K<<<B_, kBlasThreads, 0, s>>>(__VA_ARGS__);    \
+    } while (0)
 
-// f: field pointers, coef: scalars, partials: device scratch (kBlasBlocks * 4 doubles),
-// out: device result (up to 4 doubles).  Returns the number of reduced values (0 if none).
-int blas_run(int op, int prec, const Geom &g, void *const *f, const double *coef, double *partials, double *out,
-             cudaStream_t s) {
+int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail, cudaStream_t s) {
     const long Vh = g.Vh, st = g.stride;
-    const int B = kBlasBlocks, T = kBlasThreads;
     int nred = 0;
     switch (op) {
-        case 0:  // p_update(r=f0, p=f1, v=f2; beta=coef0,1, omega=coef2,3)
-            QX_PREC_SWITCH(prec, (k_p_update<P><<<B, T, 0, s>>>(Vh, st, f[0], f[1], f[2], d2(coef), d2(coef + 2))));
+        case OP_P_UPDATE:  // p = r + beta (p - omega v): r=f0, p=f1, v=f2
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_p_update<P>, Vh, st, f[0], f[1], f[2], co[0], co[1]));
             break;
-        case 1:  // caxpy: f1 += c f0
-            QX_PREC_SWITCH(prec, (k_caxpy<P><<<B, T, 0, s>>>(Vh, st, d2(coef), f[0], f[1])));
+        case OP_CAXPY:  // f1 += c f0
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_caxpy<P>, Vh, st, co[0], f[0], f[1]));
             break;
-        case 2:  // xpay: f2 = f0 + a f1
-            QX_PREC_SWITCH(prec, (k_xpay<P><<<B, T, 0, s>>>(Vh, st, f[0], coef[0], f[1], f[2])));
+        case OP_XPAY:  // f2 = f0 + a f1
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_xpay<P>, Vh, st, f[0], co[0].v.x, f[1], f[2]));
             break;
-        case 3:  // cdot(f0, f1)
-            QX_PREC_SWITCH(prec, (k_cdot<P><<<B, T, 0, s>>>(Vh, st, f[0], f[1], partials)));
+        case OP_CDOT:  // <f0, f1>
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_cdot<P>, Vh, st, f[0], f[1], tail));
             nred = 2;
             break;
-        case 4:  // norm2(f0)
-            QX_PREC_SWITCH(prec, (k_norm2<P><<<B, T, 0, s>>>(Vh, st, f[0], partials)));
+        case OP_NORM2:
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_norm2<P>, Vh, st, f[0], tail));
             nred = 1;
             break;
-        case 5:  // tdot(t=f0, s=f1)
-            QX_PREC_SWITCH(prec, (k_tdot<P><<<B, T, 0, s>>>(Vh, st, f[0], f[1], partials)));
+        case OP_TDOT:  // (<f0, f1>, |f0|^2)
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_tdot<P>, Vh, st, f[0], f[1], tail));
             nred = 3;
             break;
-        case 6:  // final(x=f0, p=f1, s=f2, t=f3, rhat=f4; alpha=c0,1 omega=c2,3)
-            QX_PREC_SWITCH(prec, (k_bicg_final<P><<<B, T, 0, s>>>(Vh, st, f[0], f[1], f[2], f[3], f[4], d2(coef), d2(coef + 2), partials)));
+        case OP_FINAL:  // x=f0, p=f1, s=f2, t=f3, rhat=f4
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bicg_final<P>, Vh, st, f[0], f[1], f[2], f[3], f[4], co[0], co[1], tail));
             nred = 3;
             break;
-        case 7:  // bmr_norm: f1 = f0 - f1
-            QX_PREC_SWITCH(prec, (k_bmr_norm<P><<<B, T, 0, s>>>(Vh, st, f[0], f[1], partials)));
+        case OP_BMR_NORM:  // f1 = f0 - f1
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bmr_norm<P>, Vh, st, f[0], f[1], tail));
             nred = 1;
             break;
         default:
             throw Error(QUDAX_ERR_ARG, "blas: bad op");
     }
     QX_CUDA(cudaGetLastError());
-    if (nred) {
-        k_reduce_final<<<1, kBlasThreads, 0, s>>>(partials, B, nred, out);
-        QX_CUDA(cudaGetLastError());
-    }
     return nred;
 }
 
 void blas_xpy_mixed(int pd, int ps, const Geom &g, const void *x, void *y, cudaStream_t s) {
-    const int B = kBlasBlocks, T = kBlasThreads;
+    const int T = kBlasThreads;
 #define QX_XM(A, C) \
-    if (pd == A && ps == C) { k_xpy_mixed<A, C><<<B, T, 0, s>>>(g.Vh, g.stride, x, y); QX_CUDA(cudaGetLastError()); return; }
+    if (pd == A && ps == C) { k_xpy_mixed<A, C><<<one_wave(k_xpy_mixed<A, C>), T, 0, s>>>(g.Vh, g.stride, x, y); QX_CUDA(cudaGetLastError()); return; }
     QX_XM(8, 8) QX_XM(8, 4) QX_XM(8, 2) QX_XM(4, 4) QX_XM(4, 2) QX_XM(2, 2) QX_XM(4, 8) QX_XM(2, 8) QX_XM(2, 4)
 #undef QX_XM
     throw Error(QUDAX_ERR_ARG, "xpy_mixed: bad precision");

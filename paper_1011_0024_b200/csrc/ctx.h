@@ -35,6 +35,16 @@ struct qudax_ctx {
     };
     std::vector<TimingRec> trecs;
     std::vector<cudaEvent_t> ev_pool;
+    // Dslash launches inside a captured CUDA graph: their (external) events are re-recorded at
+    // every replay, so they are harvested into running sums after each replay
+    std::vector<TimingRec> graph_trecs;
+    struct TimingAcc {
+        long long launches = 0, sites = 0;
+        double ms = 0, flops = 0, bytes_c = 0, bytes_p = 0;
+    } tacc[3];
+    bool capturing = false;
+    bool no_graphs = false;   // QUDAX_NO_GRAPHS=1: eager solver iterations (debug / comparison)
+    qx::SolverScalars *d_scal = nullptr, *h_scal = nullptr;
     std::vector<void *> allocs;       // device allocations owned by the ctx
     std::vector<void *> host_allocs;  // pinned host allocations
 
@@ -64,6 +74,8 @@ struct qudax_ctx {
     // workspace
     void *tmp_odd[3] = {}, *tmp_even[3] = {};
     double *partials = nullptr, *red_out = nullptr, *h_red = nullptr;
+    double *dpart = nullptr;  // per-CTA partials of Dslash-fused reductions
+    unsigned *d_counter = nullptr;  // last-CTA counter of the stream-ordered reductions
     double *stage = nullptr;  // fp64 full-slab staging (V_loc * 24 doubles)
     int *d_flag = nullptr;
 
@@ -81,13 +93,26 @@ inline int prec_idx(int prec) { return prec == 8 ? 0 : (prec == 4 ? 1 : 2); }
 void *dalloc(qudax_ctx *c, size_t bytes);
 void *halloc(qudax_ctx *c, size_t bytes);
 void check_prec(int prec);
+// optional reduction fused into a Dslash epilogue (see DslashRed); res: 3 global sums (host)
+struct RedReq {
+    int kind;
+    const void *rhat;
+    double *res;              // host results (S == nullptr), or
+    SolverScalars *S = nullptr; // device: sums land in S->red, then the recurrence coef_mode
+    int coef_mode = COEF_NONE;
+};
 void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
-               double a);
-void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger);
+               double a, const RedReq *red = nullptr, int reverse = 0);
+void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr);
+int dslash_threads();
 void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int parity, bool inverse);
 // run a BLAS op; if it reduces, globally sum and return the values in res (host)
 int blas_op(qudax_ctx *c, int op, int prec, void *const *f, const double *coef, double *res);
+void blas_op_dev(qudax_ctx *c, int op, int prec, void *const *f, const CoefArg *co, SolverScalars *S, int mode);
+void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, int mode);
 void xpy_mixed_op(qudax_ctx *c, int pd, int ps, const void *x, void *y);
 void convert_op(qudax_ctx *c, void *dst, int pd, const void *src, int ps);
 void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *p, qudax_solve_stats *st);
+void harvest_graph_timing(qudax_ctx *c);
+void release_graph_timing(qudax_ctx *c);
 }  // namespace qx

@@ -24,6 +24,7 @@
 #pragma once
 #include "core.cuh"
 #include "internal.h"
+#include "reduce.cuh"
 
 namespace qx {
 
@@ -196,11 +197,11 @@ template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) 
 #else
 #define QX_MINB_OF(P) DslashMinBlocks<P>::value
 #endif
+// one output site; red[] receives this site's contribution to the optional fused reduction
 template <int P, int RECON, bool DAG, int KIND>
-__global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
+__device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double red[3]) {
     using R = typename Prec<P>::R;
-    const int tid = blockIdx.x * blockDim.x + threadIdx.x;
-    if (tid >= a.nthreads) return;
+    if (a.reverse) tid = a.nthreads - 1 - tid;
     int i;
     if (a.range == RANGE_ALL) i = tid;
     else if (a.range == RANGE_INTERIOR) i = a.F + tid;
@@ -362,18 +363,64 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
             o[(s * 3 + c) * 2] = res[s][c].r;
             o[(s * 3 + c) * 2 + 1] = res[s][c].i;
         }
-    SpinorIO<P>::store(a.out, a.stride, i, o);
+    if (a.red_kind == RED_NONE) {
+        SpinorIO<P>::store(a.out, a.stride, i, o);
+        return;
+    }
+    // fused BiCGstab reductions over what was stored (half: the requantised values)
+    SpinorIO<P>::store_requant(a.out, a.stride, i, o);
+    R w[24];
+    SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? a.x : a.rhat, a.stride, i, w);
+#pragma unroll
+    for (int k = 0; k < 12; ++k) {
+        const double orr = o[2 * k], oi = o[2 * k + 1], wr = w[2 * k], wi = w[2 * k + 1];
+        if (a.red_kind == RED_XDOT_NORM) {  // (<out, x>, |out|^2)
+            red[0] += orr * wr + oi * wi;
+            red[1] += orr * wi - oi * wr;
+            red[2] += orr * orr + oi * oi;
+        } else {                             // <rhat, out>
+            red[0] += wr * orr + wi * oi;
+            red[1] += wr * oi - wi * orr;
+        }
+    }
+}
+
+template <int P, int RECON, bool DAG, int KIND>
+__global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
+    // one thread per output site (a one-wave grid-stride variant measured 8-25% slower: the
+    // hardware CTA scheduler balances the memory-latency-bound CTAs better than a fixed wave)
+    const int tid = blockIdx.x * blockDim.x + threadIdx.x;
+    double red[3] = {0.0, 0.0, 0.0};
+    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND>(a, tid, red);
+    if (a.red_kind != RED_NONE) reduce_with_tail<3, QX_DSLASH_THREADS>(red, a.tail);
+}
+
+template <int P, int RC, bool DG, int KD>
+int dslash_blocks(int nthreads) {
+    return (nthreads + QX_DSLASH_THREADS - 1) / QX_DSLASH_THREADS;
+}
+
+template <int P>
+int dslash_blocks_prec(int recon, int dagger, int kind, int nthreads) {
+#define QX_DB(RC, DG, KD) \
+    if (recon == RC && dagger == DG && kind == KD) return dslash_blocks<P, RC, DG, KD>(nthreads);
+#define QX_DB_K(RC, DG) QX_DB(RC, DG, 0) QX_DB(RC, DG, 1) QX_DB(RC, DG, 2)
+#define QX_DB_D(RC) QX_DB_K(RC, false) QX_DB_K(RC, true)
+    QX_DB_D(18) QX_DB_D(12) QX_DB_D(8)
+#undef QX_DB_D
+#undef QX_DB_K
+#undef QX_DB
+    throw Error(QUDAX_ERR_ARG, "dslash: unsupported recon/kind");
 }
 
 template <int P>
 void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
     const int threads = QX_DSLASH_THREADS;
-    const int blocks = (a.nthreads + threads - 1) / threads;
-    if (blocks == 0) return;
-#define QX_DS(RC, DG, KD)                                                     \
-    if (recon == RC && dagger == DG && kind == KD) {                          \
-        dslash_kernel<P, RC, DG, KD><<<blocks, threads, 0, s>>>(a);           \
-        return;                                                               \
+    if (a.nthreads <= 0) return;
+#define QX_DS(RC, DG, KD)                                                                       \
+    if (recon == RC && dagger == DG && kind == KD) {                                            \
+        dslash_kernel<P, RC, DG, KD><<<dslash_blocks<P, RC, DG, KD>(a.nthreads), threads, 0, s>>>(a); \
+        return;                                                                                 \
     }
 #define QX_DS_K(RC, DG) QX_DS(RC, DG, 0) QX_DS(RC, DG, 1) QX_DS(RC, DG, 2)
 #define QX_DS_D(RC) QX_DS_K(RC, false) QX_DS_K(RC, true)

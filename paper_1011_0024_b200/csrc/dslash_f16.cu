@@ -6,4 +6,7 @@ namespace qx {
 void launch_dslash_f16(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
     launch_dslash_prec<2>(recon, dagger, kind, a, s);
 }
+int dslash_blocks_f16(int recon, int dagger, int kind, int nthreads) {
+    return dslash_blocks_prec<2>(recon, dagger, kind, nthreads);
+}
 }  // namespace qx

@@ -6,4 +6,8 @@ namespace qx {
 void launch_dslash_f32(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
     launch_dslash_prec<4>(recon, dagger, kind, a, s);
 }
+int dslash_threads() { return QX_DSLASH_THREADS; }
+int dslash_blocks_f32(int recon, int dagger, int kind, int nthreads) {
+    return dslash_blocks_prec<4>(recon, dagger, kind, nthreads);
+}
 }  // namespace qx

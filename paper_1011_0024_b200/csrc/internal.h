@@ -67,6 +67,25 @@ struct Geom {
     long stride, fstride;  // padded Vh, padded F
 };
 
+// ----------------------------------------------------------------------------- reductions
+// device-resident BiCGstab scalars (Algorithm R), advanced by apply_coef after each reduction
+struct SolverScalars {
+    double2 rho, rho_new, alpha, malpha, omega, beta;
+    double r2;
+    double red[3];
+};
+enum CoefMode { COEF_NONE = 0, COEF_ALPHA = 1, COEF_OMEGA = 2, COEF_RHO = 3 };
+// a grid reduction with a last-CTA tail (reduce.cuh)
+struct RedTail {
+    double *partials;      // [total_blocks][nred] per-CTA sums
+    unsigned *counter;     // zero on entry, reset to zero by the last CTA
+    int total_blocks;      // CTAs contributing (all launches of this reduction)
+    int block_offset;      // this launch's first slot
+    double *out;           // totals (S->red when coef_mode != COEF_NONE)
+    SolverScalars *S;
+    int coef_mode;
+};
+
 // ----------------------------------------------------------------------------- kernels
 enum SiteRange { RANGE_ALL = 0, RANGE_INTERIOR = 1, RANGE_BOUNDARY = 2 };
 
@@ -89,11 +108,21 @@ struct DslashArgs {
     const void *clover;    // parity p: T (xpay) or T^{-1} (clover_inv)
     const void *ghost_back; // upper (non-dagger) half-spinors from rank-1, face layout
     const void *ghost_fwd;  // lower (non-dagger) half-spinors from rank+1
+    // optional fused reduction over the output (BiCGstab, P:542-558 kernel fusion)
+    int red_kind;          // RED_NONE, RED_XDOT_NORM: (<out,x>, |out|^2), RED_RHAT_DOT: <rhat,out>
+    RedTail tail;          // 3 sums per CTA; block_offset set per launch (split launches)
+    const void *rhat;
+    int reverse;           // 1: map CTAs to sites from the top of the range down (L2 reuse, see matpc)
 };
+enum DslashRed { RED_NONE = 0, RED_XDOT_NORM = 1, RED_RHAT_DOT = 2 };
 
 void launch_dslash_f64(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
 void launch_dslash_f32(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
 void launch_dslash_f16(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
+// CTAs a launch of `nthreads` sites uses (one resident wave at most)
+int dslash_blocks_f64(int recon, int dagger, int kind, int nthreads);
+int dslash_blocks_f32(int recon, int dagger, int kind, int nthreads);
+int dslash_blocks_f16(int recon, int dagger, int kind, int nthreads);
 
 // face pack: t_loc = 0 slice half (lower if !dagger) -> send_back; t_loc = T_loc-1 half
 // (upper if !dagger) -> send_fwd.  `in` is the Dslash input field (parity 1-p).
@@ -121,8 +150,18 @@ void launch_clover_apply(int prec, const Geom &g, const void *cl, const void *in
 // 6 bicgstab final update, 7 r = b - r with |r|^2.  Returns the number of reduced doubles
 // written to `out` (device).
 enum BlasOp { OP_P_UPDATE = 0, OP_CAXPY, OP_XPAY, OP_CDOT, OP_NORM2, OP_TDOT, OP_FINAL, OP_BMR_NORM };
-int blas_run(int op, int prec, const Geom &g, void *const *f, const double *coef, double *partials, double *out,
-             cudaStream_t s);
+// a BLAS coefficient: the value v, or (d != nullptr) a device scalar read by the kernel
+struct CoefArg {
+    double2 v;
+    const double2 *d;
+};
+#ifdef __CUDACC__
+__device__ __forceinline__ double2 coef_get(const CoefArg &c) { return c.d ? *c.d : c.v; }
+#endif
+// `tail` describes the reduction of reducing ops (partials/counter/out/S/coef_mode; the
+// block fields are filled in here).  Returns the number of reduced doubles (0 if none).
+int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail, cudaStream_t s);
+void launch_coef(SolverScalars *S, int mode, cudaStream_t s);
 void blas_xpy_mixed(int pd, int ps, const Geom &g, const void *x, void *y, cudaStream_t s);
 int blas_partial_blocks();
 

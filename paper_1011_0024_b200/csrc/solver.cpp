@@ -54,6 +54,40 @@ static cd cdot_of(qudax_ctx *c, int prec, void *a, void *b) {
     return cd(r[0], r[1]);
 }
 
+static SolverScalars *scalars(qudax_ctx *c) {
+    if (!c->d_scal) {
+        c->d_scal = static_cast<SolverScalars *>(dalloc(c, sizeof(SolverScalars)));
+        c->h_scal = static_cast<SolverScalars *>(halloc(c, sizeof(SolverScalars)));
+    }
+    return c->d_scal;
+}
+
+// Capture `body` (stream-ordered work on c->stream, possibly forking to the comm stream for
+// the NCCL halo) into an instantiated CUDA graph.  *nlaunch = library kernels per replay.
+template <typename F>
+static cudaGraphExec_t capture_graph(qudax_ctx *c, F &&body, long long *nlaunch) {
+    const long long l0 = c->launches;
+    c->capturing = true;
+    QX_CUDA(cudaStreamBeginCapture(c->stream, cudaStreamCaptureModeThreadLocal));
+    try {
+        body();
+    } catch (...) {
+        cudaGraph_t g;
+        cudaStreamEndCapture(c->stream, &g);
+        c->capturing = false;
+        throw;
+    }
+    cudaGraph_t graph;
+    QX_CUDA(cudaStreamEndCapture(c->stream, &graph));
+    c->capturing = false;
+    cudaGraphExec_t exec;
+    QX_CUDA(cudaGraphInstantiate(&exec, graph, 0));
+    cudaGraphDestroy(graph);
+    *nlaunch = c->launches - l0;
+    c->launches = l0;
+    return exec;
+}
+
 void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *sp, qudax_solve_stats *st) {
     QX_CHECK(c->gauge_loaded, QUDAX_ERR_STATE, "gauge not loaded");
     const int Pd = sp->prec, Ps = sp->prec_sloppy;
@@ -102,8 +136,19 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     copy(c, r0, rs, Ps);
     double rNorm = bnorm;
     double r0Norm = rNorm, maxrr = rNorm, maxrx = rNorm;
-    cd rho(1, 0), alpha(1, 0), omega(1, 0);
-    cd rho_new = cdot_of(c, Ps, r0, rs);
+    // device-resident scalars: the iteration needs no host round trip (the coefficient
+    // recurrences run in tiny kernels after each fused reduction)
+    SolverScalars *S = scalars(c);
+    SolverScalars h0{};
+    {
+        const cd rn = cdot_of(c, Ps, r0, rs);
+        h0.rho = make_double2(1, 0);
+        h0.rho_new = make_double2(rn.real(), rn.imag());
+        h0.alpha = make_double2(1, 0);
+        h0.omega = make_double2(1, 0);
+        h0.beta = make_double2(0, 0);  // first iteration: p = rs + 0 * (p - omega v) = rs
+        QX_CUDA(cudaMemcpyAsync(S, &h0, sizeof(h0), cudaMemcpyHostToDevice, c->stream));
+    }
     int k = 0, updates = 0;
     bool converged = (bnorm == 0.0);
     const double V_h_all = (double)g.Vh * g.nranks;
@@ -113,39 +158,48 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     const double matpc_flops = mm.flops * V_h_all;
     const double blas_flops_iter = 960.0 * V_h_all;  // reading Q16 (fused BLAS per iteration)
 
-    while (!converged && k < sp->maxiter) {
-        if (k == 0) {
-            copy(c, p, rs, Ps);
-        } else {
-            cd beta = (rho_new / rho) * (alpha / omega);
+    // one BiCGstab iteration, fully stream-ordered; its scalars stay on the device
+    auto enqueue_iteration = [&] {
+        {
             void *f[3] = {rs, p, v};
-            double co[4] = {beta.real(), beta.imag(), omega.real(), omega.imag()};
-            blas_op(c, OP_P_UPDATE, Ps, f, co, nullptr);
+            CoefArg co[2] = {{{0, 0}, &S->beta}, {{0, 0}, &S->omega}};
+            blas_op_dev(c, OP_P_UPDATE, Ps, f, co, S, COEF_NONE);      // p = r + beta (p - omega v)
         }
-        matpc_op(c, v, p, Ps, 0);
-        cd r0v = cdot_of(c, Ps, r0, v);
-        alpha = rho_new / r0v;
+        RedReq red_rv{RED_RHAT_DOT, r0, nullptr, S, COEF_ALPHA};
+        matpc_op(c, v, p, Ps, 0, &red_rv);                            // v = Mhat p; alpha = rho'/<rhat0,v>
         {
             void *f[2] = {v, rs};
-            double co[2] = {-alpha.real(), -alpha.imag()};
-            blas_op(c, OP_CAXPY, Ps, f, co, nullptr);
+            CoefArg co[1] = {{{0, 0}, &S->malpha}};
+            blas_op_dev(c, OP_CAXPY, Ps, f, co, S, COEF_NONE);         // s = r - alpha v
         }
-        matpc_op(c, t, rs, Ps, 0);
-        double td[3];
-        {
-            void *f[2] = {t, rs};
-            blas_op(c, OP_TDOT, Ps, f, nullptr, td);
-        }
-        omega = cd(td[0], td[1]) / td[2];
-        double fin[3];
+        RedReq red_ts{RED_XDOT_NORM, nullptr, nullptr, S, COEF_OMEGA};
+        matpc_op(c, t, rs, Ps, 0, &red_ts);                            // t = Mhat s; omega = <t,s>/|t|^2
         {
             void *f[5] = {xs, p, rs, t, r0};
-            double co[4] = {alpha.real(), alpha.imag(), omega.real(), omega.imag()};
-            blas_op(c, OP_FINAL, Ps, f, co, fin);
+            CoefArg co[2] = {{{0, 0}, &S->alpha}, {{0, 0}, &S->omega}};
+            blas_op_dev(c, OP_FINAL, Ps, f, co, S, COEF_RHO);          // x += a p + w s; r = s - w t; rho', beta
         }
-        rho = rho_new;
-        rho_new = cd(fin[1], fin[2]);
-        rNorm = std::sqrt(fin[0]);
+        QX_CUDA(cudaMemcpyAsync(c->h_scal, S, sizeof(SolverScalars), cudaMemcpyDeviceToHost, c->stream));
+    };
+    // Replay the iteration as one CUDA graph (no per-kernel launch latency, no host syncs
+    // inside the iteration).  Not possible with the host transport (its hooks run on the host).
+    const bool use_graph = (c->comm != QUDAX_COMM_HOST) && !c->no_graphs;
+    cudaGraphExec_t gexec = nullptr;
+    long long graph_launches = 0;
+
+    while (!converged && k < sp->maxiter) {
+        if (!use_graph || k == 0) {
+            enqueue_iteration();  // the first iteration runs eagerly (allocates lazily-created buffers)
+        } else {
+            if (!gexec) gexec = capture_graph(c, enqueue_iteration, &graph_launches);
+            QX_CUDA(cudaGraphLaunch(gexec, c->stream));
+            c->launches += graph_launches;
+        }
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        harvest_graph_timing(c);
+        const SolverScalars &hs = *c->h_scal;
+        double rNorm_it = std::sqrt(hs.r2);
+        rNorm = rNorm_it;
         ++k;
         flops += 2 * matpc_flops + blas_flops_iter;
         if (rNorm > maxrx) maxrx = rNorm;
@@ -170,12 +224,23 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
                 r0Norm = rNorm;
                 maxrx = rNorm;
             }
-            rho_new = cdot_of(c, Ps, r0, rs);
+            // continue the recurrences from the replaced residual: rho' = <rhat0, r>,
+            // beta = (rho'/rho)(alpha/omega) with the iteration's rho, alpha, omega
+            const cd rn = cdot_of(c, Ps, r0, rs);
+            const cd rho(hs.rho.x, hs.rho.y), al(hs.alpha.x, hs.alpha.y), om(hs.omega.x, hs.omega.y);
+            const cd beta = (rn / rho) * (al / om);
+            SolverScalars upd = hs;
+            upd.rho_new = make_double2(rn.real(), rn.imag());
+            upd.beta = make_double2(beta.real(), beta.imag());
+            QX_CUDA(cudaMemcpyAsync(S, &upd, sizeof(upd), cudaMemcpyHostToDevice, c->stream));
+            QX_CUDA(cudaStreamSynchronize(c->stream));
             ++updates;
             if (rNorm <= stop) converged = true;
         }
         if (sp->res_history && k - 1 < sp->history_cap) sp->res_history[k - 1] = bnorm > 0 ? rNorm / bnorm : 0.0;
     }
+    if (gexec) cudaGraphExecDestroy(gexec);
+    release_graph_timing(c);
     st->iters = k;
     st->reliable_updates = updates;
     st->true_res_schur = bnorm > 0 ? rNorm / bnorm : 0.0;
