@@ -245,6 +245,14 @@ qudax_status qudax_solve_bicgstab(qudax_ctx *ctx, double *host_x, const double *
 qudax_status qudax_solve_bicgstab_dev(qudax_ctx *ctx, double *dev_x, const double *dev_b,
                                       const qudax_solve_param *p, qudax_solve_stats *st);
 
+/* CGNR ("Conjugate Gradients [7] on the normal equations"): CG on
+ * Mhat^dag Mhat x_e = Mhat^dag bhat in precision p->prec (prec_sloppy and delta ignored), with
+ * the same Schur prepare / reconstruct and the same TRUE-residual stopping test as BiCGstab. */
+qudax_status qudax_solve_cgnr(qudax_ctx *ctx, double *host_x, const double *host_b,
+                              const qudax_solve_param *p, qudax_solve_stats *st);
+qudax_status qudax_solve_cgnr_dev(qudax_ctx *ctx, double *dev_x, const double *dev_b,
+                                  const qudax_solve_param *p, qudax_solve_stats *st);
+
 #ifdef __cplusplus
 }
 #endif

@@ -606,6 +606,7 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         QX_CHECK(g.V < (1L << 30), QUDAX_ERR_ARG, "local volume too large for 32-bit site indexing");
         c->device = p->device;
         if (const char *ng = std::getenv("QUDAX_NO_GRAPHS")) c->no_graphs = (ng[0] == '1');
+        if (const char *fg = std::getenv("QUDAX_GRAPHS")) c->force_graphs = (fg[0] == '1');
         c->comm = p->comm;
         c->overlap = p->overlap;
         c->dev_alloc = p->dev_alloc; c->dev_free = p->dev_free; c->alloc_user = p->alloc_user;
@@ -847,13 +848,18 @@ qudax_status qudax_cdot(qudax_ctx *c, const void *a, const void *b, int prec, do
     });
 }
 
-qudax_status qudax_solve_bicgstab_dev(qudax_ctx *c, double *x, const double *b, const qudax_solve_param *p,
-                                      qudax_solve_stats *st) {
+}  // extern "C"
+
+namespace {
+using SolveFn = void (*)(qudax_ctx *, double *, const double *, const qudax_solve_param *, qudax_solve_stats *);
+
+qudax_status solve_device_entry(SolveFn fn, qudax_ctx *c, double *x, const double *b, const qudax_solve_param *p,
+                                qudax_solve_stats *st) {
     if (!c) return QUDAX_ERR_ARG;
     qudax_status s = guard(c, [&] {
         QX_CHECK(x && b && p && st, QUDAX_ERR_ARG, "solve: null argument");
         auto t0 = std::chrono::steady_clock::now();
-        solve_dev(c, x, b, p, st);
+        fn(c, x, b, p, st);
         st->secs = std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
         st->gflops = st->flops / st->secs * 1e-9;
     });
@@ -861,8 +867,9 @@ qudax_status qudax_solve_bicgstab_dev(qudax_ctx *c, double *x, const double *b, 
     return s;
 }
 
-qudax_status qudax_solve_bicgstab(qudax_ctx *c, double *host_x, const double *host_b, const qudax_solve_param *p,
-                                  qudax_solve_stats *st) {
+// host buffers: H2D of b and D2H of x are inside the call (and its timing)
+qudax_status solve_host_entry(SolveFn fn, qudax_ctx *c, double *host_x, const double *host_b,
+                              const qudax_solve_param *p, qudax_solve_stats *st) {
     if (!c) return QUDAX_ERR_ARG;
     double *db = nullptr, *dx = nullptr;
     auto t0 = std::chrono::steady_clock::now();
@@ -872,7 +879,7 @@ qudax_status qudax_solve_bicgstab(qudax_ctx *c, double *host_x, const double *ho
         db = static_cast<double *>(dalloc(c, n));
         dx = static_cast<double *>(dalloc(c, n));
         QX_CUDA(cudaMemcpyAsync(db, host_b, n, cudaMemcpyHostToDevice, c->stream));
-        solve_dev(c, dx, db, p, st);
+        fn(c, dx, db, p, st);
         QX_CUDA(cudaMemcpyAsync(host_x, dx, n, cudaMemcpyDeviceToHost, c->stream));
         QX_CUDA(cudaStreamSynchronize(c->stream));
         dfree(c, db);
@@ -885,6 +892,26 @@ qudax_status qudax_solve_bicgstab(qudax_ctx *c, double *host_x, const double *ho
     if (dx) dfree(c, dx);
     if (s == QUDAX_OK && p->tol > 0 && st->true_res > p->tol * (1 + 1e-3)) return QUDAX_ERR_NOT_CONVERGED;
     return s;
+}
+}  // namespace
+
+extern "C" {
+
+qudax_status qudax_solve_bicgstab_dev(qudax_ctx *c, double *x, const double *b, const qudax_solve_param *p,
+                                      qudax_solve_stats *st) {
+    return solve_device_entry(solve_dev, c, x, b, p, st);
+}
+qudax_status qudax_solve_bicgstab(qudax_ctx *c, double *host_x, const double *host_b, const qudax_solve_param *p,
+                                  qudax_solve_stats *st) {
+    return solve_host_entry(solve_dev, c, host_x, host_b, p, st);
+}
+qudax_status qudax_solve_cgnr_dev(qudax_ctx *c, double *x, const double *b, const qudax_solve_param *p,
+                                  qudax_solve_stats *st) {
+    return solve_device_entry(cgnr_dev, c, x, b, p, st);
+}
+qudax_status qudax_solve_cgnr(qudax_ctx *c, double *host_x, const double *host_b, const qudax_solve_param *p,
+                              qudax_solve_stats *st) {
+    return solve_host_entry(cgnr_dev, c, host_x, host_b, p, st);
 }
 
 }  // extern "C"

@@ -44,6 +44,7 @@ struct qudax_ctx {
     } tacc[3];
     bool capturing = false;
     bool no_graphs = false;   // QUDAX_NO_GRAPHS=1: eager solver iterations (debug / comparison)
+    bool force_graphs = false;  // QUDAX_GRAPHS=1: graph replay also with nranks > 1
     qx::SolverScalars *d_scal = nullptr, *h_scal = nullptr;
     std::vector<void *> allocs;       // device allocations owned by the ctx
     std::vector<void *> host_allocs;  // pinned host allocations
@@ -85,7 +86,7 @@ struct qudax_ctx {
         void *b_e = nullptr, *b_o = nullptr, *bh = nullptr, *x_e = nullptr, *x_o = nullptr, *r = nullptr, *t_e = nullptr,
              *t_o = nullptr;
         void *rs = nullptr, *xs = nullptr, *p = nullptr, *v = nullptr, *t = nullptr, *r0 = nullptr;
-    } sws;
+    } sws, cgws;
 };
 
 namespace qx {
@@ -113,6 +114,7 @@ void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, in
 void xpy_mixed_op(qudax_ctx *c, int pd, int ps, const void *x, void *y);
 void convert_op(qudax_ctx *c, void *dst, int pd, const void *src, int ps);
 void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *p, qudax_solve_stats *st);
+void cgnr_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *p, qudax_solve_stats *st);
 void harvest_graph_timing(qudax_ctx *c);
 void release_graph_timing(qudax_ctx *c);
 }  // namespace qx

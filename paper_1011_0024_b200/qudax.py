@@ -127,6 +127,8 @@ SIGNATURES = {
     "qudax_cdot": ([_P, _P, _P, _I, _DP], _I),
     "qudax_solve_bicgstab": ([_P, _DP, _DP, ctypes.POINTER(SolveParam), ctypes.POINTER(SolveStats)], _I),
     "qudax_solve_bicgstab_dev": ([_P, _P, _P, ctypes.POINTER(SolveParam), ctypes.POINTER(SolveStats)], _I),
+    "qudax_solve_cgnr": ([_P, _DP, _DP, ctypes.POINTER(SolveParam), ctypes.POINTER(SolveStats)], _I),
+    "qudax_solve_cgnr_dev": ([_P, _P, _P, ctypes.POINTER(SolveParam), ctypes.POINTER(SolveStats)], _I),
 }
 
 
@@ -380,6 +382,18 @@ class Context:
             sp.res_history = history.ctypes.data_as(_DP)
             sp.history_cap = int(history.size)
         return sp
+
+    def solve_cgnr(self, b, tol=1e-10, maxiter=10000, prec=DOUBLE, use_schur=True, allow_not_converged=False,
+                   history=None):
+        """CGNR on Mhat^dag Mhat in one precision; host arrays as in solve()."""
+        b = np.ascontiguousarray(b, dtype=np.complex128)
+        x = np.zeros_like(b)
+        sp = self._solve_param(tol, 0.0, maxiter, prec, prec, use_schur, history)
+        st = SolveStats()
+        rc = lib().qudax_solve_cgnr(self._h, _dptr(x), _dptr(b), ctypes.byref(sp), ctypes.byref(st))
+        if rc and not (allow_not_converged and rc == 6):
+            self._check(rc)
+        return x, st.as_dict()
 
     def solve(self, b, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
               allow_not_converged=False, history=None, out=None):

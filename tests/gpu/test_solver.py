@@ -80,3 +80,37 @@ def test_solver_fixed_iterations_and_device_entry(torch_cuda, system):
     res = np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b)
     assert abs(res - st["true_res"]) < 1e-9
     ctx.close()
+
+
+def test_loopback_solve_matches_unsplit(torch_cuda, system):
+    """The solver through the split halo path (NCCL loopback at N=1, CUDA-graph replay with the
+    NCCL p2p inside) reproduces the unsplit solve: the exchange moves bits only; only the
+    grouping of the fused reductions' partial sums differs (interior/boundary CTAs)."""
+    U, wc = system
+    b = qgen.point_source(DIMS, 1, 0)
+    xs = []
+    for comm in (qudax.COMM_NONE, qudax.COMM_NCCL):
+        ctx = qudax.Context(DIMS, comm=comm, nccl_id=qudax.nccl_unique_id() if comm else None)
+        ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+        x, st = ctx.solve(b, tol=1e-10, delta=0.1, maxiter=2000, prec=8, prec_sloppy=4)
+        xs.append((x, st["iters"]))
+        ctx.close()
+    assert abs(xs[0][1] - xs[1][1]) <= 1
+    assert np.linalg.norm(xs[0][0] - xs[1][0]) / np.linalg.norm(xs[0][0]) < 1e-8
+
+
+@pytest.mark.parametrize("prec,recon,tol", [(8, 18, 1e-12), (4, 12, 1e-5)])
+def test_cgnr_vs_oracle(torch_cuda, system, prec, recon, tol):
+    """CGNR on the normal equations: the oracle's fp64 true
+    residual of the solution meets tol; the solution agrees with the oracle's BiCGstab one."""
+    U, wc = system
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=prec, recon=recon, t_boundary=-1)
+    b = qgen.point_source(DIMS, 0, 2)
+    x, st = ctx.solve_cgnr(b, tol=tol, maxiter=5000, prec=prec)
+    res = np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b)
+    print("cgnr", prec, st["iters"], st["true_res"], res)
+    assert res <= tol * (1.5 if prec == 4 else 1.001)
+    if prec == 8:
+        assert abs(res - st["true_res"]) <= 1e-9
+    ctx.close()
