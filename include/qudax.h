@@ -230,6 +230,15 @@ qudax_status qudax_dslash(qudax_ctx *ctx, void *out, const void *in, const void 
                           int out_parity, int dagger, int kind, double a);
 /* out_e = Mhat in_e (dagger = 0) or Mhat^dag in_e (dagger = 1); 2 Dslash kernels + 2 halos. */
 qudax_status qudax_matpc(qudax_ctx *ctx, void *out, const void *in, int prec, int dagger);
+/* Multi-RHS forms (the paper's production calls the solver for many
+ * right-hand sides per configuration): nrhs (1..8) independent fields
+ * in one launch that streams the links and clover from HBM about once for all of them.
+ * Arrays of nrhs device field pointers; x may be NULL unless kind = CLOVER_XPAY.  Results are
+ * bitwise those of nrhs single calls.  Partitioned contexts apply the single-RHS path per field. */
+qudax_status qudax_dslash_multi(qudax_ctx *ctx, void *const *out, const void *const *in, const void *const *x,
+                                int nrhs, int prec, int out_parity, int dagger, int kind, double a);
+qudax_status qudax_matpc_multi(qudax_ctx *ctx, void *const *out, const void *const *in, int nrhs, int prec,
+                               int dagger);
 /* out_e = Mhat^dag Mhat in_e (the CGNR normal operator). */
 qudax_status qudax_mdagm(qudax_ctx *ctx, void *out, const void *in, int prec);
 

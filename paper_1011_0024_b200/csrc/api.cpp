@@ -147,7 +147,7 @@ static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int
         launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
         return;
     }
-    qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads};
+    qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads, a.nrhs > 1 ? a.nrhs : 1};
     if (c->capturing) {  // graph: external event-record nodes, re-recorded at each replay
         QX_CUDA(cudaEventRecordWithFlags(r.a, c->stream, cudaEventRecordExternal));
         launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
@@ -161,19 +161,33 @@ static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int
     c->trecs.push_back(r);
 }
 
+// totals of one recorded launch: flops and bytes over its sites and right-hand sides (links and
+// clover are compulsory once per site, spinor reads/writes once per site and RHS)
+static void rec_model(const qudax_ctx::TimingRec &r, qudax_site_model *out) {
+    qudax_site_model m, hop;
+    qudax_model(r.prec, r.recon, r.kind, &m);
+    const double w = r.prec, nrm = (r.prec == 2) ? 4 : 0;
+    const double sp = 24 * w + nrm;
+    const double per_rhs = (r.kind == QUDAX_CLOVER_XPAY ? 3 : 2) * sp;  // in, out (, x)
+    (void)hop;
+    out->flops = m.flops * r.sites * r.nrhs;
+    out->bytes_compulsory = ((m.bytes_compulsory - per_rhs) + per_rhs * r.nrhs) * r.sites;
+    out->bytes_paper = m.bytes_paper * r.sites * r.nrhs;
+}
+
 void harvest_graph_timing(qudax_ctx *c) {
     for (auto &r : c->graph_trecs) {
         float ms = 0;
         QX_CUDA(cudaEventElapsedTime(&ms, r.a, r.b));
         qudax_site_model m;
-        qudax_model(r.prec, r.recon, r.kind, &m);
+        rec_model(r, &m);
         auto &t = c->tacc[prec_idx(r.prec)];
         t.launches += 1;
-        t.sites += r.sites;
+        t.sites += r.sites * r.nrhs;
         t.ms += ms;
-        t.flops += m.flops * r.sites;
-        t.bytes_c += m.bytes_compulsory * r.sites;
-        t.bytes_p += m.bytes_paper * r.sites;
+        t.flops += m.flops;
+        t.bytes_c += m.bytes_compulsory;
+        t.bytes_p += m.bytes_paper;
     }
 }
 
@@ -185,14 +199,9 @@ void release_graph_timing(qudax_ctx *c) {
     c->graph_trecs.clear();
 }
 
-void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
-               double a, const RedReq *red, int reverse) {
-    check_prec(prec);
-    QX_CHECK(p == 0 || p == 1, QUDAX_ERR_ARG, "parity must be 0 or 1");
-    QX_CHECK(kind >= 0 && kind <= 2, QUDAX_ERR_ARG, "bad dslash kind");
-    QX_CHECK(out && in && (kind != QUDAX_CLOVER_XPAY || x), QUDAX_ERR_ARG, "null field");
-    QX_CHECK(out != in, QUDAX_ERR_ARG, "dslash cannot run in place");
-    auto &gc = gauge_for(c, prec);
+// kernel arguments common to every Dslash launch of (precision, output parity, kind)
+static DslashArgs base_args(qudax_ctx *c, const qudax_ctx::GaugeCopy &gc, int prec, int p, int kind, double a,
+                            int reverse) {
     const Geom &g = c->g;
     DslashArgs args{};
     args.X = g.X; args.Y = g.Y; args.Z = g.Z; args.T_loc = g.T_loc; args.Xh = g.Xh;
@@ -203,7 +212,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     args.bc_back = (g.rank == 0) ? (double)c->t_bc : 1.0;
     args.a = a;
     args.reverse = reverse;
-    args.in = in; args.out = out; args.x = x;
+    args.nrhs = 1;
     for (int m = 0; m < 4; ++m)
         for (int q = 0; q < 2; ++q) args.gauge[m][q] = gc.d[m][q];
     args.gauge_ghost = gc.ghost[1 - p];
@@ -212,6 +221,20 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         QX_CHECK(cl.valid, QUDAX_ERR_STATE, "no clover in this precision");
         args.clover = (kind == QUDAX_CLOVER_XPAY) ? cl.T[p] : cl.Tinv[p];
     }
+    return args;
+}
+
+void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
+               double a, const RedReq *red, int reverse) {
+    check_prec(prec);
+    QX_CHECK(p == 0 || p == 1, QUDAX_ERR_ARG, "parity must be 0 or 1");
+    QX_CHECK(kind >= 0 && kind <= 2, QUDAX_ERR_ARG, "bad dslash kind");
+    QX_CHECK(out && in && (kind != QUDAX_CLOVER_XPAY || x), QUDAX_ERR_ARG, "null field");
+    QX_CHECK(out != in, QUDAX_ERR_ARG, "dslash cannot run in place");
+    auto &gc = gauge_for(c, prec);
+    const Geom &g = c->g;
+    DslashArgs args = base_args(c, gc, prec, p, kind, a, reverse);
+    args.in = in; args.out = out; args.x = x;
     int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
     const int TPB = dslash_threads();
     const bool split = (c->comm == QUDAX_COMM_NCCL && c->overlap && g.T_loc > 2);
@@ -299,6 +322,52 @@ void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, con
     // the second kernel walks the lattice top-down: the timeslices the first kernel touched
     // last (their links, T^{-1} D in and the dirty tmp lines) are still in the 126 MB L2
     dslash_op(c, out, t, in, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, red, 1);
+}
+
+// Multi-RHS Dslash (SURVEY NEXT row 2, P:748-753 / P:1092-1094: many right-hand sides per
+// configuration): one launch for n fields, consecutive CTAs taking the same sites for
+// different RHS so the links and clover are read from HBM about once for all of them.
+// Partitioned runs (halo exchange per RHS) apply the single-RHS path per field.
+void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, const void *const *x, int n, int prec,
+                     int p, int dagger, int kind, double a, int reverse) {
+    check_prec(prec);
+    QX_CHECK(n >= 1 && n <= kMaxRhs, QUDAX_ERR_ARG, "nrhs must be 1.." + std::to_string(kMaxRhs));
+    QX_CHECK(p == 0 || p == 1, QUDAX_ERR_ARG, "parity must be 0 or 1");
+    QX_CHECK(kind >= 0 && kind <= 2, QUDAX_ERR_ARG, "bad dslash kind");
+    for (int k = 0; k < n; ++k) {
+        QX_CHECK(out[k] && in[k] && (kind != QUDAX_CLOVER_XPAY || (x && x[k])), QUDAX_ERR_ARG, "null field");
+        QX_CHECK(out[k] != in[k], QUDAX_ERR_ARG, "dslash cannot run in place");
+    }
+    if (c->comm != QUDAX_COMM_NONE || n == 1) {
+        for (int k = 0; k < n; ++k)
+            dslash_op(c, out[k], in[k], x ? x[k] : nullptr, prec, p, dagger, kind, a, nullptr, reverse);
+        return;
+    }
+    auto &gc = gauge_for(c, prec);
+    DslashArgs args = base_args(c, gc, prec, p, kind, a, reverse);
+    args.nrhs = n;
+    for (int k = 0; k < n; ++k) {
+        args.in_m[k] = in[k];
+        args.out_m[k] = out[k];
+        args.x_m[k] = x ? x[k] : nullptr;
+    }
+    args.ghosted = 0;
+    args.range = RANGE_ALL;
+    args.nthreads = (int)c->g.Vh;
+    launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
+    c->launches += 1;
+}
+
+void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger) {
+    QX_CHECK(n >= 1 && n <= kMaxRhs, QUDAX_ERR_ARG, "nrhs must be 1.." + std::to_string(kMaxRhs));
+    void *t[kMaxRhs];
+    for (int k = 0; k < n; ++k) {
+        auto &slot = c->tmp_multi[prec_idx(prec)][k];
+        if (!slot) slot = dalloc(c, spinor_bytes(prec, c->g.stride));
+        t[k] = slot;
+    }
+    dslash_multi_op(c, t, in, nullptr, n, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, 0);
+    dslash_multi_op(c, out, t, in, n, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, 1);
 }
 
 void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int parity, bool inverse) {
@@ -708,13 +777,13 @@ qudax_status qudax_get_kernel_stats(qudax_ctx *c, int prec_filter, qudax_kernel_
             float ms = 0;
             QX_CUDA(cudaEventElapsedTime(&ms, r.a, r.b));
             qudax_site_model m;
-            qudax_model(r.prec, r.recon, r.kind, &m);
+            rec_model(r, &m);
             o->launches += 1;
             o->ms_total += ms;
-            o->sites += r.sites;
-            o->flops += m.flops * r.sites;
-            o->bytes_compulsory += m.bytes_compulsory * r.sites;
-            o->bytes_paper += m.bytes_paper * r.sites;
+            o->sites += r.sites * r.nrhs;
+            o->flops += m.flops;
+            o->bytes_compulsory += m.bytes_compulsory;
+            o->bytes_paper += m.bytes_paper;
         }
         for (int q = 0; q < 3; ++q) {
             const int pr = q == 0 ? 8 : (q == 1 ? 4 : 2);
@@ -807,6 +876,24 @@ qudax_status qudax_dslash(qudax_ctx *c, void *out, const void *in, const void *x
                           int dagger, int kind, double a) {
     if (!c) return QUDAX_ERR_ARG;
     return guard(c, [&] { dslash_op(c, out, in, x, prec, out_parity, dagger ? 1 : 0, kind, a); });
+}
+
+qudax_status qudax_dslash_multi(qudax_ctx *c, void *const *out, const void *const *in, const void *const *x,
+                                int nrhs, int prec, int out_parity, int dagger, int kind, double a) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        QX_CHECK(out && in, QUDAX_ERR_ARG, "dslash_multi: null arrays");
+        dslash_multi_op(c, out, in, x, nrhs, prec, out_parity, dagger ? 1 : 0, kind, a, 0);
+    });
+}
+
+qudax_status qudax_matpc_multi(qudax_ctx *c, void *const *out, const void *const *in, int nrhs, int prec,
+                               int dagger) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        QX_CHECK(out && in, QUDAX_ERR_ARG, "matpc_multi: null arrays");
+        matpc_multi_op(c, out, in, nrhs, prec, dagger ? 1 : 0);
+    });
 }
 
 qudax_status qudax_matpc(qudax_ctx *c, void *out, const void *in, int prec, int dagger) {

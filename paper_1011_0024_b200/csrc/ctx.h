@@ -32,6 +32,7 @@ struct qudax_ctx {
         cudaEvent_t a, b;
         int prec, recon, kind;
         long sites;
+        int nrhs = 1;  // multi-RHS launch: links and clover are compulsory once, spinors per RHS
     };
     std::vector<TimingRec> trecs;
     std::vector<cudaEvent_t> ev_pool;
@@ -74,6 +75,7 @@ struct qudax_ctx {
 
     // workspace
     void *tmp_odd[3] = {}, *tmp_even[3] = {};
+    void *tmp_multi[3][qx::kMaxRhs] = {};
     double *partials = nullptr, *red_out = nullptr, *h_red = nullptr;
     double *dpart = nullptr;  // per-CTA partials of Dslash-fused reductions
     unsigned *d_counter = nullptr;  // last-CTA counter of the stream-ordered reductions
@@ -105,6 +107,9 @@ struct RedReq {
 void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
                double a, const RedReq *red = nullptr, int reverse = 0);
 void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr);
+void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, const void *const *x, int n, int prec,
+                     int p, int dagger, int kind, double a, int reverse);
+void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger);
 int dslash_threads();
 void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int parity, bool inverse);
 // run a BLAS op; if it reduces, globally sum and return the values in res (host)

@@ -199,7 +199,8 @@ template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) 
 #endif
 // one output site; red[] receives this site's contribution to the optional fused reduction
 template <int P, int RECON, bool DAG, int KIND>
-__device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double red[3]) {
+__device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin, void *fout, const void *fx, int tid,
+                                            double red[3]) {
     using R = typename Prec<P>::R;
     if (a.reverse) tid = a.nthreads - 1 - tid;
     int i;
@@ -228,7 +229,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double
     if (xpay_early) {
         R v[24];
         Cx<R> xs[4][3];
-        SpinorIO<P>::load(a.x, a.stride, i, v);
+        SpinorIO<P>::load(fx, a.stride, i, v);
         unpack_spinor(v, xs);
         apply_clover<P>(a.clover, a.stride, i, xs, acc);
         const R inv_a = (R)(1.0 / a.a);
@@ -252,11 +253,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double
         const int nb = (x == 0 ? lex + (X - 1) : lex - 1) >> 1;
         R v[24];
         Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::load(a.in, a.stride, nf, v);
+        SpinorIO<P>::load(fin, a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[0][p], a.stride, i, u);
         spatial_hop<0, SF, false>(ps, u, (R)1, acc);
-        SpinorIO<P>::load(a.in, a.stride, nb, v);
+        SpinorIO<P>::load(fin, a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[0][op], a.stride, nb, u);
         spatial_hop<0, SB, true>(ps, u, (R)1, acc);
@@ -267,11 +268,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double
         const int nb = (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1;
         R v[24];
         Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::load(a.in, a.stride, nf, v);
+        SpinorIO<P>::load(fin, a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[1][p], a.stride, i, u);
         spatial_hop<1, SF, false>(ps, u, (R)1, acc);
-        SpinorIO<P>::load(a.in, a.stride, nb, v);
+        SpinorIO<P>::load(fin, a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[1][op], a.stride, nb, u);
         spatial_hop<1, SB, true>(ps, u, (R)1, acc);
@@ -282,11 +283,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double
         const int nb = (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1;
         R v[24];
         Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::load(a.in, a.stride, nf, v);
+        SpinorIO<P>::load(fin, a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[2][p], a.stride, i, u);
         spatial_hop<2, SF, false>(ps, u, (R)1, acc);
-        SpinorIO<P>::load(a.in, a.stride, nb, v);
+        SpinorIO<P>::load(fin, a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[2][op], a.stride, nb, u);
         spatial_hop<2, SB, true>(ps, u, (R)1, acc);
@@ -304,10 +305,10 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double
             if (a.ghosted) {
                 FaceIO<P>::load(a.ghost_fwd, a.fstride, i - t * a.F, h);
             } else {
-                SpinorIO<P>::load_half(a.in, a.stride, (lex - (T_loc - 1) * XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
+                SpinorIO<P>::load_half(fin, a.stride, (lex - (T_loc - 1) * XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
             }
         } else {
-            SpinorIO<P>::load_half(a.in, a.stride, (lex + XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
+            SpinorIO<P>::load_half(fin, a.stride, (lex + XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
         }
         LinkIO<P, RECON>::load(a.gauge[3][p], a.stride, i, u);
         temporal_hop<FWD_UPPER, false>(h, u, cf, acc);
@@ -322,12 +323,12 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double
                 LinkIO<P, RECON>::load(a.gauge_ghost, a.fstride, i, u);
             } else {
                 const int nb = (lex + (T_loc - 1) * XYZ) >> 1;
-                SpinorIO<P>::load_half(a.in, a.stride, nb, BWD_UPPER ? 0 : 1, h);
+                SpinorIO<P>::load_half(fin, a.stride, nb, BWD_UPPER ? 0 : 1, h);
                 LinkIO<P, RECON>::load(a.gauge[3][op], a.stride, nb, u);
             }
         } else {
             const int nb = (lex - XYZ) >> 1;
-            SpinorIO<P>::load_half(a.in, a.stride, nb, BWD_UPPER ? 0 : 1, h);
+            SpinorIO<P>::load_half(fin, a.stride, nb, BWD_UPPER ? 0 : 1, h);
             LinkIO<P, RECON>::load(a.gauge[3][op], a.stride, nb, u);
         }
         temporal_hop<BWD_UPPER, true>(h, u, cb, acc);
@@ -351,7 +352,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double
     } else {  // a == 0: out = T x
         R v[24];
         Cx<R> xs[4][3];
-        SpinorIO<P>::load(a.x, a.stride, i, v);
+        SpinorIO<P>::load(fx, a.stride, i, v);
         unpack_spinor(v, xs);
         apply_clover<P>(a.clover, a.stride, i, xs, res);
     }
@@ -364,13 +365,13 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, int tid, double
             o[(s * 3 + c) * 2 + 1] = res[s][c].i;
         }
     if (a.red_kind == RED_NONE) {
-        SpinorIO<P>::store(a.out, a.stride, i, o);
+        SpinorIO<P>::store(fout, a.stride, i, o);
         return;
     }
     // fused BiCGstab reductions over what was stored (half: the requantised values)
-    SpinorIO<P>::store_requant(a.out, a.stride, i, o);
+    SpinorIO<P>::store_requant(fout, a.stride, i, o);
     R w[24];
-    SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? a.x : a.rhat, a.stride, i, w);
+    SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx : a.rhat, a.stride, i, w);
 #pragma unroll
     for (int k = 0; k < 12; ++k) {
         const double orr = o[2 * k], oi = o[2 * k + 1], wr = w[2 * k], wi = w[2 * k + 1];
@@ -389,9 +390,19 @@ template <int P, int RECON, bool DAG, int KIND>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
     // one thread per output site (a one-wave grid-stride variant measured 8-25% slower: the
     // hardware CTA scheduler balances the memory-latency-bound CTAs better than a fixed wave)
-    const int tid = blockIdx.x * blockDim.x + threadIdx.x;
+    // multi-RHS (a.nrhs > 1): consecutive CTAs take the same sites for different right-hand
+    // sides, so the links and clover they stream are served from L2 after the first of them
+    int blk = blockIdx.x, rhs = 0;
+    if (a.nrhs > 1) {
+        rhs = blk % a.nrhs;
+        blk /= a.nrhs;
+    }
+    const int tid = blk * blockDim.x + threadIdx.x;
     double red[3] = {0.0, 0.0, 0.0};
-    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND>(a, tid, red);
+    const void *fin = a.nrhs > 1 ? a.in_m[rhs] : a.in;
+    void *fout = a.nrhs > 1 ? a.out_m[rhs] : a.out;
+    const void *fx = a.nrhs > 1 ? a.x_m[rhs] : a.x;
+    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND>(a, fin, fout, fx, tid, red);
     if (a.red_kind != RED_NONE) reduce_with_tail<3, QX_DSLASH_THREADS>(red, a.tail);
 }
 
@@ -419,7 +430,8 @@ void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cu
     if (a.nthreads <= 0) return;
 #define QX_DS(RC, DG, KD)                                                                       \
     if (recon == RC && dagger == DG && kind == KD) {                                            \
-        dslash_kernel<P, RC, DG, KD><<<dslash_blocks<P, RC, DG, KD>(a.nthreads), threads, 0, s>>>(a); \
+        dslash_kernel<P, RC, DG, KD><<<dslash_blocks<P, RC, DG, KD>(a.nthreads) * (a.nrhs > 1 ? a.nrhs : 1), \
+                                       threads, 0, s>>>(a);                                     \
         return;                                                                                 \
     }
 #define QX_DS_K(RC, DG) QX_DS(RC, DG, 0) QX_DS(RC, DG, 1) QX_DS(RC, DG, 2)

@@ -88,6 +88,7 @@ struct RedTail {
 
 // ----------------------------------------------------------------------------- kernels
 enum SiteRange { RANGE_ALL = 0, RANGE_INTERIOR = 1, RANGE_BOUNDARY = 2 };
+constexpr int kMaxRhs = 8;
 
 struct DslashArgs {
     // geometry
@@ -113,6 +114,11 @@ struct DslashArgs {
     RedTail tail;          // 3 sums per CTA; block_offset set per launch (split launches)
     const void *rhat;
     int reverse;           // 1: map CTAs to sites from the top of the range down (L2 reuse, see matpc)
+    // multi-RHS launch: nrhs > 1 uses in_m / out_m / x_m instead of in/out/x
+    int nrhs;
+    const void *in_m[kMaxRhs];
+    void *out_m[kMaxRhs];
+    const void *x_m[kMaxRhs];
 };
 enum DslashRed { RED_NONE = 0, RED_XDOT_NORM = 1, RED_RHAT_DOT = 2 };
 

@@ -122,6 +122,8 @@ SIGNATURES = {
     "qudax_spinor_convert": ([_P, _P, _I, _P, _I], _I),
     "qudax_dslash": ([_P, _P, _P, _P, _I, _I, _I, _I, _D], _I),
     "qudax_matpc": ([_P, _P, _P, _I, _I], _I),
+    "qudax_dslash_multi": ([_P, ctypes.POINTER(_P), ctypes.POINTER(_P), ctypes.POINTER(_P), _I, _I, _I, _I, _I, _D], _I),
+    "qudax_matpc_multi": ([_P, ctypes.POINTER(_P), ctypes.POINTER(_P), _I, _I, _I], _I),
     "qudax_mdagm": ([_P, _P, _P, _I], _I),
     "qudax_norm2": ([_P, _P, _I, _DP], _I),
     "qudax_cdot": ([_P, _P, _P, _I, _DP], _I),
@@ -360,6 +362,19 @@ class Context:
 
     def matpc(self, out, inp, prec, dagger=False):
         self._check(lib().qudax_matpc(self._h, out.data_ptr(), inp.data_ptr(), int(prec), int(bool(dagger))))
+
+    @staticmethod
+    def _ptrs(fields):
+        return (_P * len(fields))(*[f.data_ptr() for f in fields])
+
+    def dslash_multi(self, outs, ins, prec, out_parity, dagger=False, kind=HOP, xs=None, a=0.0):
+        xp = self._ptrs(xs) if xs is not None else None
+        self._check(lib().qudax_dslash_multi(self._h, self._ptrs(outs), self._ptrs(ins), xp, len(ins), int(prec),
+                                             int(out_parity), int(bool(dagger)), int(kind), float(a)))
+
+    def matpc_multi(self, outs, ins, prec, dagger=False):
+        self._check(lib().qudax_matpc_multi(self._h, self._ptrs(outs), self._ptrs(ins), len(ins), int(prec),
+                                            int(bool(dagger))))
 
     def mdagm(self, out, inp, prec):
         self._check(lib().qudax_mdagm(self._h, out.data_ptr(), inp.data_ptr(), int(prec)))

@@ -27,6 +27,7 @@ def main():
     ap.add_argument("--reps", type=int, default=50)
     ap.add_argument("--cases", default="f32-12,h-12,f64-18")
     ap.add_argument("--tag", default=os.environ.get("QUDAX_LIB", "default"))
+    ap.add_argument("--nrhs", default="", help="comma list: also time multi-RHS Mhat for these counts")
     args = ap.parse_args()
     dims = tuple(int(v) for v in args.dims.split(","))
     peak = json.load(open(os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))),
@@ -52,6 +53,22 @@ def main():
             gbs = ks["bytes_compulsory"] / (ks["ms_total"] * 1e-3) * 1e-9
             res[name] = {"us": 1e3 * ks["ms_total"] / ks["launches"], "GBs": round(gbs, 1),
                          "frac": round(gbs / peak, 4), "GFLOPS": round(ks["flops"] / (ks["ms_total"] * 1e-3) * 1e-9, 1)}
+        for n in [int(v) for v in args.nrhs.split(",") if v]:
+            ins = [ctx.new_field(prec) for _ in range(n)]
+            outs = [ctx.new_field(prec) for _ in range(n)]
+            for f in ins:
+                ctx.spinor_load(f, prec, 0, psi)
+            for _ in range(3):
+                ctx.matpc_multi(outs, ins, prec)
+            ctx.kernel_timing(True)
+            for _ in range(max(5, args.reps // n)):
+                ctx.matpc_multi(outs, ins, prec)
+            ks = ctx.kernel_stats()
+            ctx.kernel_timing(False)
+            gbs = ks["bytes_compulsory"] / (ks["ms_total"] * 1e-3) * 1e-9
+            res[f"matpc_x{n}"] = {"us_per_rhs": 1e3 * ks["ms_total"] / (ks["launches"] / 2) / n,
+                                  "GFLOPS": round(ks["flops"] / (ks["ms_total"] * 1e-3) * 1e-9, 1),
+                                  "GBs_multi_model": round(gbs, 1), "frac": round(gbs / peak, 4)}
         print(json.dumps(res), flush=True)
     ctx.close()
 
