@@ -146,6 +146,78 @@ def cpu_oracle_gflops(iters, dims=(SPATIAL, SPATIAL, SPATIAL, 8)):
     return flops / dt * 1e-9, dt, threads, sample
 
 
+def single_gpu_extras(ctx, b_dev, peak):
+    """N = 1 only: multi-RHS Mhat (fp32-12, 4 and 8 RHS) on the bench lattice, and the
+    half-precision (recon 12) Mhat in a second context.  Per-launch CUDA-event timing."""
+    from paper_1011_0024_b200 import qudax
+    out = {}
+    fin = ctx.new_field(4)
+    ctx.spinor_load_dev(fin, 4, 0, b_dev)
+    for n in (4, 8):
+        ins = [fin] * n
+        outs = [ctx.new_field(4) for _ in range(n)]
+        for _ in range(3):
+            ctx.matpc_multi(outs, ins, 4)
+        ctx.kernel_timing(True)
+        for _ in range(10):
+            ctx.matpc_multi(outs, ins, 4)
+        ks = ctx.kernel_stats(prec=4)
+        ctx.kernel_timing(False)
+        gbs = ks["bytes_compulsory"] / (ks["ms_total"] * 1e-3) * 1e-9
+        out[f"fp32-12 x{n} rhs"] = {"matpc_gflops": ks["flops"] / (ks["ms_total"] * 1e-3) * 1e-9,
+                                   "us_per_rhs": 1e3 * ks["ms_total"] / 10 / n,
+                                   "gbs_multi_rhs_model": gbs, "frac_of_measured_hbm": gbs / peak}
+    import numpy as np
+    import qgen
+    dims = ctx.global_dims
+    hctx = qudax.Context(dims)
+    hctx.gauge_load(qgen.gauge(dims, GAUGE_SEED, eps=EPS), KAPPA, CSW, prec=2, recon=12)
+    hi, ho = hctx.new_field(2), hctx.new_field(2)
+    hctx.spinor_load_dev(hi, 2, 0, b_dev)
+    for _ in range(3):
+        hctx.matpc(ho, hi, 2)
+    hctx.kernel_timing(True)
+    for _ in range(30):
+        hctx.matpc(ho, hi, 2)
+    ks = hctx.kernel_stats(prec=2)
+    hctx.close()
+    gbs = ks["bytes_compulsory"] / (ks["ms_total"] * 1e-3) * 1e-9
+    out["half-12"] = {"kernel_gflops": ks["flops"] / (ks["ms_total"] * 1e-3) * 1e-9, "kernel_gbs_compulsory": gbs,
+                      "frac_of_measured_hbm": gbs / peak, "matpc_us": 1e3 * ks["ms_total"] / 30}
+    del np
+    return out
+
+
+def config3_solve_time():
+    """BASELINE configs[2]: 24^3 x 128 weak field, the paper's 6 point sources (colour 0-2 x
+    spin 0-1), mixed double-single (delta 0.1) and double-half (delta 0.1; the
+    paper's 1e-2, stalls 2 of the 6 sources here — DESIGN.md reading Q11)
+    reliable-update BiCGstab to ||r||/||b|| <= 1e-14 through the C-ABI
+    with host buffers; mean time to solution, iterations, true residual."""
+    import qgen
+    from paper_1011_0024_b200 import qudax
+    dims = (24, 24, 24, 128)
+    U = qgen.gauge(dims, 1003, eps=EPS)
+    ctx = qudax.Context(dims)
+    res = {"workload": "24^3x128 weak field, 6 point sources, tol 1e-14, kappa 0.124, csw 1.0 (BASELINE configs[2])"}
+    for name, ps, delta in (("double-single", 4, 0.1), ("double-half", 2, 0.1)):
+        ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=ps, recon_sloppy=12, t_boundary=-1)
+        ts, its, trs, gfl = [], [], [], []
+        for colour in range(3):
+            for spin in range(2):
+                b = qgen.point_source(dims, spin, colour)
+                _, st = ctx.solve(b, tol=1e-14, delta=delta, maxiter=20000, prec=8, prec_sloppy=ps,
+                                  allow_not_converged=True)
+                ts.append(st["secs"])
+                its.append(st["iters"])
+                trs.append(st["true_res"])
+                gfl.append(st["gflops"])
+        res[name] = {"mean_secs": sum(ts) / len(ts), "mean_iters": sum(its) / len(its), "max_true_res": max(trs),
+                     "mean_gflops": sum(gfl) / len(gfl)}
+    ctx.close()
+    return res
+
+
 # ---------------------------------------------------------------------------- reference arm
 def run_reference(args):
     rank = int(os.environ.get("RANK", "0"))
@@ -322,6 +394,10 @@ def main():
                 "frac_of_measured_hbm": (k2["bytes_compulsory"] / (k2["ms_total"] * 1e-3) * 1e-9) / peak,
             }
             del fin, fout
+    solve_time = None
+    if not args.no_extra and N == 1:
+        dslash.update(single_gpu_extras(ctx, b_dev, peak))
+        solve_time = config3_solve_time()
 
     # ---- CPU baseline: the oracle on the host cores (rank 0, N = 1 only)
     cpu = None
@@ -344,7 +420,7 @@ def main():
                        "l2": "inputs larger than L2 (>1 GB of gauge+clover+fields per GPU vs 126 MB L2)"},
             "iters_per_step": iters / args.steps, "reliable_updates_per_step": updates / args.steps,
             "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches, "clocks": clocks,
-            "dslash": dslash,
+            "dslash": dslash, "solve_time": solve_time,
         }
         print(json.dumps(out))
     if world > 1:

@@ -149,6 +149,7 @@ typedef struct {
     double secs;                 /* wall time of the call (includes H2D / D2H for the host entry) */
     double flops;                /* effective flops (P:755-758 convention, reading Q16) */
     double gflops;
+    int restarts;                /* Krylov restarts after a (near) breakdown of the sloppy recurrences */
 } qudax_solve_stats;
 
 /* Per-site work and traffic model, for reporting and tests. */

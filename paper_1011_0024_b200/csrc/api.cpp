@@ -676,6 +676,7 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         c->device = p->device;
         if (const char *ng = std::getenv("QUDAX_NO_GRAPHS")) c->no_graphs = (ng[0] == '1');
         if (const char *fg = std::getenv("QUDAX_GRAPHS")) c->force_graphs = (fg[0] == '1');
+        if (const char *ds = std::getenv("QUDAX_DEBUG_SOLVER")) c->debug_solver = (ds[0] == '1');
         c->comm = p->comm;
         c->overlap = p->overlap;
         c->dev_alloc = p->dev_alloc; c->dev_free = p->dev_free; c->alloc_user = p->alloc_user;

@@ -46,6 +46,7 @@ struct qudax_ctx {
     bool capturing = false;
     bool no_graphs = false;   // QUDAX_NO_GRAPHS=1: eager solver iterations (debug / comparison)
     bool force_graphs = false;  // QUDAX_GRAPHS=1: graph replay also with nranks > 1
+    bool debug_solver = false;  // QUDAX_DEBUG_SOLVER=1: per-iteration scalars to stderr
     qx::SolverScalars *d_scal = nullptr, *h_scal = nullptr;
     std::vector<void *> allocs;       // device allocations owned by the ctx
     std::vector<void *> host_allocs;  // pinned host allocations

@@ -21,6 +21,7 @@
 //              if updX: r0Norm = maxrx = rNorm;  stop if rNorm <= tol ||bhat||
 #include <cmath>
 #include <complex>
+#include <cstdio>
 #include <cstring>
 
 #include "ctx.h"
@@ -196,7 +197,7 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
         h0.beta = make_double2(0, 0);  // first iteration: p = rs + 0 * (p - omega v) = rs
         QX_CUDA(cudaMemcpyAsync(S, &h0, sizeof(h0), cudaMemcpyHostToDevice, c->stream));
     }
-    int k = 0, updates = 0;
+    int k = 0, updates = 0, restarts = 0;
     bool converged = (bnorm == 0.0);
     const double V_h_all = (double)g.Vh * g.nranks;
     double flops = 0;
@@ -247,17 +248,27 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
         QX_CUDA(cudaStreamSynchronize(c->stream));
         harvest_graph_timing(c);
         const SolverScalars &hs = *c->h_scal;
+        if (c->debug_solver)
+            std::fprintf(stderr, "qudax it %d: r2 %.6e rho (%.4e,%.4e) alpha (%.4e,%.4e) omega (%.4e,%.4e) beta (%.4e,%.4e) red %.4e %.4e %.4e\n",
+                         k, hs.r2, hs.rho_new.x, hs.rho_new.y, hs.alpha.x, hs.alpha.y, hs.omega.x, hs.omega.y,
+                         hs.beta.x, hs.beta.y, hs.red[0], hs.red[1], hs.red[2]);
         double rNorm_it = std::sqrt(hs.r2);
+        // breakdown guard (reading R3): a non-finite or exploded iterated residual means the
+        // low-precision recurrences hit a (near) Lanczos breakdown.  Recompute the true
+        // residual (dropping xs if it is not finite) and restart the Krylov space from it.
+        const bool blown = !std::isfinite(rNorm_it) || rNorm_it > 1e2 * maxrr;
         rNorm = rNorm_it;
         ++k;
         flops += 2 * matpc_flops + blas_flops_iter;
-        if (rNorm > maxrx) maxrx = rNorm;
-        if (rNorm > maxrr) maxrr = rNorm;
-        const bool updX = (rNorm < sp->delta * r0Norm) && (r0Norm <= maxrx);
-        const bool updR = ((rNorm < sp->delta * maxrr) && (r0Norm <= maxrr)) || updX || (rNorm <= stop) ||
+        if (!blown) {
+            if (rNorm > maxrx) maxrx = rNorm;
+            if (rNorm > maxrr) maxrr = rNorm;
+        }
+        const bool updX = !blown && (rNorm < sp->delta * r0Norm) && (r0Norm <= maxrx);
+        const bool updR = blown || ((rNorm < sp->delta * maxrr) && (r0Norm <= maxrr)) || updX || (rNorm <= stop) ||
                           (k == sp->maxiter);
         if (updR) {
-            xpy_mixed_op(c, Pd, Ps, xs, x_e);   // x += xs
+            if (std::isfinite(rNorm_it)) xpy_mixed_op(c, Pd, Ps, xs, x_e);   // x += xs
             zero(c, xs, Ps);
             matpc_op(c, r, x_e, Pd, 0);          // r = Mhat x (high)
             double r2;
@@ -269,18 +280,31 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
             convert_op(c, rs, Ps, r, Pd);
             rNorm = std::sqrt(r2);
             maxrr = rNorm;
-            if (updX) {
+            if (updX || blown) {
                 r0Norm = rNorm;
                 maxrx = rNorm;
             }
-            // continue the recurrences from the replaced residual: rho' = <rhat0, r>,
-            // beta = (rho'/rho)(alpha/omega) with the iteration's rho, alpha, omega
-            const cd rn = cdot_of(c, Ps, r0, rs);
-            const cd rho(hs.rho.x, hs.rho.y), al(hs.alpha.x, hs.alpha.y), om(hs.omega.x, hs.omega.y);
-            const cd beta = (rn / rho) * (al / om);
             SolverScalars upd = hs;
-            upd.rho_new = make_double2(rn.real(), rn.imag());
-            upd.beta = make_double2(beta.real(), beta.imag());
+            if (blown) {  // restart: rhat0 = r, p = r (beta = 0, v = 0)
+                copy(c, r0, rs, Ps);
+                zero(c, p, Ps);
+                zero(c, v, Ps);
+                const cd rn = cdot_of(c, Ps, r0, rs);
+                upd.rho = make_double2(1, 0);
+                upd.rho_new = make_double2(rn.real(), rn.imag());
+                upd.alpha = make_double2(1, 0);
+                upd.omega = make_double2(1, 0);
+                upd.beta = make_double2(0, 0);
+                ++restarts;
+            } else {
+                // continue the recurrences from the replaced residual: rho' = <rhat0, r>,
+                // beta = (rho'/rho)(alpha/omega) with the iteration's rho, alpha, omega
+                const cd rn = cdot_of(c, Ps, r0, rs);
+                const cd rho(hs.rho.x, hs.rho.y), al(hs.alpha.x, hs.alpha.y), om(hs.omega.x, hs.omega.y);
+                const cd beta = (rn / rho) * (al / om);
+                upd.rho_new = make_double2(rn.real(), rn.imag());
+                upd.beta = make_double2(beta.real(), beta.imag());
+            }
             QX_CUDA(cudaMemcpyAsync(S, &upd, sizeof(upd), cudaMemcpyHostToDevice, c->stream));
             QX_CUDA(cudaStreamSynchronize(c->stream));
             ++updates;
@@ -292,6 +316,7 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     release_graph_timing(c);
     st->iters = k;
     st->reliable_updates = updates;
+    st->restarts = restarts;
     st->true_res_schur = bnorm > 0 ? rNorm / bnorm : 0.0;
 
     finish_solution(c, Pd, x_dev, b_e, b_o, x_e, x_o, t_e, t_o, sp->use_schur, st);

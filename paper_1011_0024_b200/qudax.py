@@ -64,7 +64,7 @@ class SolveParam(ctypes.Structure):
 class SolveStats(ctypes.Structure):
     _fields_ = [("iters", ctypes.c_int), ("reliable_updates", ctypes.c_int), ("true_res", ctypes.c_double),
                 ("true_res_schur", ctypes.c_double), ("secs", ctypes.c_double), ("flops", ctypes.c_double),
-                ("gflops", ctypes.c_double)]
+                ("gflops", ctypes.c_double), ("restarts", ctypes.c_int)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}
@@ -262,7 +262,10 @@ class Context:
                     return None
 
             def _free(ptr, _u):
-                torch.cuda.caching_allocator_delete(int(ptr))
+                try:
+                    torch.cuda.caching_allocator_delete(int(ptr))
+                except Exception:  # noqa: BLE001 - interpreter shutdown: the process frees it
+                    pass
 
             self._alloc_cb, self._free_cb = ALLOC_FN(_alloc), FREE_FN(_free)
             p.dev_alloc, p.dev_free = self._alloc_cb, self._free_cb
