@@ -184,7 +184,9 @@ const char *qudax_status_string(int status);
 /* Partition bookkeeping of rank `rank` of `nranks`. */
 qudax_status qudax_partition_info(const int global_dims[4], int nranks, int rank, qudax_partition *out);
 /* Site model for one Dslash kernel of `kind` (flops: 1320 + 504 clover + 48 xpay, Q16), or for
- * the whole Mhat when kind = -1 (3696 flops / 2976 bytes at fp32 recon 12). */
+ * the whole Mhat when kind = -1 (3696 flops / 2976 bytes at fp32 recon 12), or for
+ * the single-launch (fused) Mhat when kind = -2 (compulsory bytes: links once, T and T^{-1},
+ * input, output and the intermediate written once). */
 qudax_status qudax_model(int prec, int recon, int kind, qudax_site_model *out);
 /* ncclGetUniqueId into out[128] (rank 0 calls, caller broadcasts). */
 qudax_status qudax_nccl_unique_id(void *out128);

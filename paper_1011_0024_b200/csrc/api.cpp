@@ -316,8 +316,91 @@ static void *tmp_even(qudax_ctx *c, int prec) {
 }
 
 // Mhat = T_ee - kappa^2 D_eo T_oo^{-1} D_oe (asymmetric Schur form on even sites)
+// dispense order of the fused Mhat wavefront (matpc_fused.cuh): A(0..L), then A(k) followed
+// by B(k-L), then the remaining B's; B(0) last (it needs A(T-1) through the periodic wrap).
+static const int *fused_stages(qudax_ctx *c) {
+    if (c->fstages) return c->fstages;
+    const int T = c->g.T_loc;
+    const char *lag = std::getenv("QUDAX_FUSED_LAG");
+    const int L = lag ? std::max(1, std::atoi(lag)) : 1;
+    std::vector<int> st;
+    for (int k = 0; k <= std::min(L, T - 1); ++k) st.push_back(k);
+    std::vector<bool> bdone(T, false);
+    for (int k = L + 1; k < T; ++k) {
+        st.push_back(k);
+        const int b = k - L;
+        if (b >= 1) { st.push_back(T + b); bdone[b] = true; }
+    }
+    for (int b = 1; b < T; ++b)
+        if (!bdone[b]) st.push_back(T + b);
+    st.push_back(T + 0);
+    QX_CHECK((int)st.size() == 2 * T, QUDAX_ERR_STATE, "fused stage table");
+    int *d = static_cast<int *>(dalloc(c, sizeof(int) * st.size()));
+    QX_CUDA(cudaMemcpy(d, st.data(), sizeof(int) * st.size(), cudaMemcpyHostToDevice));
+    c->fcounters = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * (T + 1)));
+    c->fstages = d;
+    return d;
+}
+
+// Mhat as one persistent wavefront launch (unpartitioned contexts)
+static void matpc_fused(qudax_ctx *c, void *out, const void *in, void *t, int prec, int dagger, const RedReq *red) {
+    auto &gc = gauge_for(c, prec);
+    const Geom &g = c->g;
+    const int TPB = dslash_threads();
+    FusedArgs f{};
+    f.A = base_args(c, gc, prec, 1, QUDAX_CLOVER_INV, 0.0, 0);
+    f.A.in = in; f.A.out = t; f.A.ghosted = 0; f.A.range = RANGE_ALL; f.A.nthreads = (int)g.Vh;
+    f.B = base_args(c, gc, prec, 0, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, 0);
+    f.B.in = t; f.B.x = in; f.B.out = out; f.B.ghosted = 0; f.B.range = RANGE_ALL; f.B.nthreads = (int)g.Vh;
+    f.chunks = (int)((g.F + TPB - 1) / TPB);
+    f.total_items = 2 * g.T_loc * f.chunks;
+    f.stages = fused_stages(c);
+    f.work = c->fcounters;
+    f.doneA = c->fcounters + 1;
+    const int wave = prec == 8 ? matpc_fused_wave_f64(gc.recon, dagger)
+                               : (prec == 4 ? matpc_fused_wave_f32(gc.recon, dagger) : matpc_fused_wave_f16(gc.recon, dagger));
+    const int grid = std::min(wave, f.total_items);
+    if (red) {
+        QX_CHECK(red->kind == RED_RHAT_DOT ? red->rhat != nullptr : red->kind == RED_XDOT_NORM, QUDAX_ERR_ARG,
+                 "fused matpc: bad reduction");
+        if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / TPB) + 64)));
+        f.B.red_kind = red->kind;
+        f.B.rhat = red->rhat;
+        f.B.tail.partials = c->dpart;
+        f.B.tail.counter = c->d_counter;
+        f.B.tail.total_blocks = grid;
+        f.B.tail.block_offset = 0;
+        f.B.tail.out = red->S ? red->S->red : c->red_out;
+        f.B.tail.S = red->S;
+        f.B.tail.coef_mode = red->S ? red->coef_mode : COEF_NONE;
+    }
+    QX_CUDA(cudaMemsetAsync(c->fcounters, 0, sizeof(unsigned) * (g.T_loc + 1), c->stream));
+    auto launch = [&] {
+        if (prec == 8) launch_matpc_fused_f64(gc.recon, dagger, f, grid, c->stream);
+        else if (prec == 4) launch_matpc_fused_f32(gc.recon, dagger, f, grid, c->stream);
+        else launch_matpc_fused_f16(gc.recon, dagger, f, grid, c->stream);
+        QX_CUDA(cudaGetLastError());
+    };
+    if (c->timing) {
+        qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, gc.recon, -2, (long)g.Vh, 1};
+        const unsigned fl = c->capturing ? cudaEventRecordExternal : cudaEventRecordDefault;
+        QX_CUDA(cudaEventRecordWithFlags(r.a, c->stream, fl));
+        launch();
+        QX_CUDA(cudaEventRecordWithFlags(r.b, c->stream, fl));
+        (c->capturing ? c->graph_trecs : c->trecs).push_back(r);
+    } else {
+        launch();
+    }
+    c->launches += 1;
+    if (red && !red->S) global_sum(c, c->red_out, 3, red->res);
+}
+
 void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red) {
     void *t = tmp_odd(c, prec);
+    if (c->comm == QUDAX_COMM_NONE && c->fused && c->g.T_loc >= 2) {
+        matpc_fused(c, out, in, t, prec, dagger, red);
+        return;
+    }
     dslash_op(c, t, in, nullptr, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, nullptr);
     // the second kernel walks the lattice top-down: the timeslices the first kernel touched
     // last (their links, T^{-1} D in and the dirty tmp lines) are still in the 126 MB L2
@@ -618,7 +701,7 @@ qudax_status qudax_partition_info(const int global_dims[4], int nranks, int rank
 }
 
 qudax_status qudax_model(int prec, int recon, int kind, qudax_site_model *o) {
-    if (!o || (prec != 2 && prec != 4 && prec != 8) || (recon != 18 && recon != 12 && recon != 8) || kind < -1 ||
+    if (!o || (prec != 2 && prec != 4 && prec != 8) || (recon != 18 && recon != 12 && recon != 8) || kind < -2 ||
         kind > 2)
         return QUDAX_ERR_ARG;
     const double w = prec;
@@ -640,6 +723,11 @@ qudax_status qudax_model(int prec, int recon, int kind, qudax_site_model *o) {
         o->flops = a.flops + b.flops;
         o->bytes_paper = a.bytes_paper + b.bytes_paper;
         o->bytes_compulsory = a.bytes_compulsory + b.bytes_compulsory;
+        if (kind == -2) {
+            // single-launch (fused) Mhat: the links are compulsory once, both clover terms,
+            // the input (also the xpay x), the output, and the intermediate written once
+            o->bytes_compulsory = 8 * link + 2 * clov + 3 * sp;
+        }
     }
     return QUDAX_OK;
 }
@@ -677,6 +765,7 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         if (const char *ng = std::getenv("QUDAX_NO_GRAPHS")) c->no_graphs = (ng[0] == '1');
         if (const char *fg = std::getenv("QUDAX_GRAPHS")) c->force_graphs = (fg[0] == '1');
         if (const char *ds = std::getenv("QUDAX_DEBUG_SOLVER")) c->debug_solver = (ds[0] == '1');
+        if (const char *fu = std::getenv("QUDAX_FUSED")) c->fused = (fu[0] == '1');
         c->comm = p->comm;
         c->overlap = p->overlap;
         c->dev_alloc = p->dev_alloc; c->dev_free = p->dev_free; c->alloc_user = p->alloc_user;

@@ -72,16 +72,20 @@ __device__ __forceinline__ short2 ld_stream(const short2 *p) {
 // ----------------------------------------------------------------------------- SoA access
 // Load reals [4*b0, 4*(b0+nb)) (fp32/half) or [2*b0, 2*(b0+nb)) (fp64) of site i.
 // `stream` selects the no-L1-allocate path (links, clover) vs the read-only cached path.
-template <int P, int NB, bool STREAM>
+// load modes: 0 = read-only path (L1-cached, non-coherent), 1 = streamed (no L1 allocation),
+// 2 = L2 only (coherent with writes made by other CTAs earlier in the same kernel)
+template <typename V> __device__ __forceinline__ V ld_mode2(const V *p) { return __ldcg(p); }
+template <int P, int NB, int STREAM>
 struct Blocks;
 
-template <int NB, bool STREAM>
+template <int NB, int STREAM>
 struct Blocks<8, NB, STREAM> {
     static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, double *out) {
         const double2 *p = reinterpret_cast<const double2 *>(base);
 #pragma unroll
         for (int k = 0; k < NB; ++k) {
-            double2 v = STREAM ? ld_stream(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
+            double2 v = STREAM == 1 ? ld_stream(p + (b0 + k) * stride + i)
+                        : (STREAM == 2 ? __ldcg(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i));
             out[2 * k] = v.x;
             out[2 * k + 1] = v.y;
         }
@@ -93,13 +97,14 @@ struct Blocks<8, NB, STREAM> {
     }
 };
 
-template <int NB, bool STREAM>
+template <int NB, int STREAM>
 struct Blocks<4, NB, STREAM> {
     static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out) {
         const float4 *p = reinterpret_cast<const float4 *>(base);
 #pragma unroll
         for (int k = 0; k < NB; ++k) {
-            float4 v = STREAM ? ld_stream(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
+            float4 v = STREAM == 1 ? ld_stream(p + (b0 + k) * stride + i)
+                       : (STREAM == 2 ? __ldcg(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i));
             out[4 * k] = v.x;
             out[4 * k + 1] = v.y;
             out[4 * k + 2] = v.z;
@@ -143,14 +148,15 @@ __device__ __forceinline__ uint2 ld_stream_u2(const uint2 *p) {
 }
 
 // half: raw integer values scaled by `scale` (norm/32767 for spinors, 1/32767 for links)
-template <int NB, bool STREAM>
+template <int NB, int STREAM>
 struct Blocks<2, NB, STREAM> {
     static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out,
                                                 float scale) {
         const uint2 *p = reinterpret_cast<const uint2 *>(base);
 #pragma unroll
         for (int k = 0; k < NB; ++k) {
-            uint2 v = STREAM ? ld_stream_u2(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
+            uint2 v = STREAM == 1 ? ld_stream_u2(p + (b0 + k) * stride + i)
+                      : (STREAM == 2 ? __ldcg(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i));
             out[4 * k] = __fmul_rn(scale, i16lo_to_f32(v.x));
             out[4 * k + 1] = __fmul_rn(scale, i16hi_to_f32(v.x));
             out[4 * k + 2] = __fmul_rn(scale, i16lo_to_f32(v.y));
@@ -191,17 +197,20 @@ struct SpinorIO {
     }
 
     // half = 0: reals 0..11 (spins 0,1), half = 1: reals 12..23 (spins 2,3)
+    // MODE 0: read-only path; MODE 2: L2-coherent (data written earlier in the same kernel)
+    template <int MODE = 0>
     static __device__ __forceinline__ void load_half(const void *base, long stride, long i, int half, R *out) {
         if constexpr (P == 2) {
-            float nrm = __ldg(norms(base, stride) + i);
-            Blocks<2, 3, false>::load(base, stride, i, 3 * half, out, nrm * kHalfInv);
+            float nrm = MODE == 2 ? __ldcg(norms(base, stride) + i) : __ldg(norms(base, stride) + i);
+            Blocks<2, 3, MODE>::load(base, stride, i, 3 * half, out, nrm * kHalfInv);
         } else {
-            Blocks<P, BPH, false>::load(base, stride, i, BPH * half, out);
+            Blocks<P, BPH, MODE>::load(base, stride, i, BPH * half, out);
         }
     }
+    template <int MODE = 0>
     static __device__ __forceinline__ void load(const void *base, long stride, long i, R *out) {
-        load_half(base, stride, i, 0, out);
-        load_half(base, stride, i, 1, out + 12);
+        load_half<MODE>(base, stride, i, 0, out);
+        load_half<MODE>(base, stride, i, 1, out + 12);
     }
     static __device__ __forceinline__ void store(void *base, long stride, long i, const R *in) {
         if constexpr (P == 2) {

@@ -47,6 +47,12 @@ struct qudax_ctx {
     bool no_graphs = false;   // QUDAX_NO_GRAPHS=1: eager solver iterations (debug / comparison)
     bool force_graphs = false;  // QUDAX_GRAPHS=1: graph replay also with nranks > 1
     bool debug_solver = false;  // QUDAX_DEBUG_SOLVER=1: per-iteration scalars to stderr
+    // single-launch wavefront Mhat on unpartitioned contexts (QUDAX_FUSED=1).  Off by default:
+    // measured slower than the two kernels (L2 kept only ~1/3 of the reusable bytes, plus
+    // dependency waits) — profiles/r01_fused_matpc.md
+    bool fused = false;
+    const int *fstages = nullptr;
+    unsigned *fcounters = nullptr;
     qx::SolverScalars *d_scal = nullptr, *h_scal = nullptr;
     std::vector<void *> allocs;       // device allocations owned by the ctx
     std::vector<void *> host_allocs;  // pinned host allocations

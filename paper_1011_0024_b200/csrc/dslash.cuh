@@ -198,7 +198,9 @@ template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) 
 #define QX_MINB_OF(P) DslashMinBlocks<P>::value
 #endif
 // one output site; red[] receives this site's contribution to the optional fused reduction
-template <int P, int RECON, bool DAG, int KIND>
+// INMODE: load mode of the neighbour spinors (0 read-only path; 2 L2-coherent, for inputs
+// written by other CTAs earlier in the same launch — the fused Mhat kernel)
+template <int P, int RECON, bool DAG, int KIND, int INMODE = 0>
 __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin, void *fout, const void *fx, int tid,
                                             double red[3]) {
     using R = typename Prec<P>::R;
@@ -253,11 +255,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         const int nb = (x == 0 ? lex + (X - 1) : lex - 1) >> 1;
         R v[24];
         Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::load(fin, a.stride, nf, v);
+        SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[0][p], a.stride, i, u);
         spatial_hop<0, SF, false>(ps, u, (R)1, acc);
-        SpinorIO<P>::load(fin, a.stride, nb, v);
+        SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[0][op], a.stride, nb, u);
         spatial_hop<0, SB, true>(ps, u, (R)1, acc);
@@ -268,11 +270,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         const int nb = (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1;
         R v[24];
         Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::load(fin, a.stride, nf, v);
+        SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[1][p], a.stride, i, u);
         spatial_hop<1, SF, false>(ps, u, (R)1, acc);
-        SpinorIO<P>::load(fin, a.stride, nb, v);
+        SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[1][op], a.stride, nb, u);
         spatial_hop<1, SB, true>(ps, u, (R)1, acc);
@@ -283,11 +285,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         const int nb = (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1;
         R v[24];
         Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::load(fin, a.stride, nf, v);
+        SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[2][p], a.stride, i, u);
         spatial_hop<2, SF, false>(ps, u, (R)1, acc);
-        SpinorIO<P>::load(fin, a.stride, nb, v);
+        SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[2][op], a.stride, nb, u);
         spatial_hop<2, SB, true>(ps, u, (R)1, acc);
@@ -305,10 +307,10 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             if (a.ghosted) {
                 FaceIO<P>::load(a.ghost_fwd, a.fstride, i - t * a.F, h);
             } else {
-                SpinorIO<P>::load_half(fin, a.stride, (lex - (T_loc - 1) * XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
+                SpinorIO<P>::template load_half<INMODE>(fin,a.stride, (lex - (T_loc - 1) * XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
             }
         } else {
-            SpinorIO<P>::load_half(fin, a.stride, (lex + XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
+            SpinorIO<P>::template load_half<INMODE>(fin,a.stride, (lex + XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
         }
         LinkIO<P, RECON>::load(a.gauge[3][p], a.stride, i, u);
         temporal_hop<FWD_UPPER, false>(h, u, cf, acc);
@@ -323,12 +325,12 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
                 LinkIO<P, RECON>::load(a.gauge_ghost, a.fstride, i, u);
             } else {
                 const int nb = (lex + (T_loc - 1) * XYZ) >> 1;
-                SpinorIO<P>::load_half(fin, a.stride, nb, BWD_UPPER ? 0 : 1, h);
+                SpinorIO<P>::template load_half<INMODE>(fin,a.stride, nb, BWD_UPPER ? 0 : 1, h);
                 LinkIO<P, RECON>::load(a.gauge[3][op], a.stride, nb, u);
             }
         } else {
             const int nb = (lex - XYZ) >> 1;
-            SpinorIO<P>::load_half(fin, a.stride, nb, BWD_UPPER ? 0 : 1, h);
+            SpinorIO<P>::template load_half<INMODE>(fin,a.stride, nb, BWD_UPPER ? 0 : 1, h);
             LinkIO<P, RECON>::load(a.gauge[3][op], a.stride, nb, u);
         }
         temporal_hop<BWD_UPPER, true>(h, u, cb, acc);

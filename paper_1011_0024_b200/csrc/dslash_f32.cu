@@ -1,6 +1,7 @@
 // dslash_f32.cu — instantiation of the Dslash kernel family for storage precision 4 bytes/real
 // (split per precision so the 18 variants per precision compile in parallel).
 #include "dslash.cuh"
+#include "matpc_fused.cuh"
 
 namespace qx {
 void launch_dslash_f32(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
@@ -10,4 +11,8 @@ int dslash_threads() { return QX_DSLASH_THREADS; }
 int dslash_blocks_f32(int recon, int dagger, int kind, int nthreads) {
     return dslash_blocks_prec<4>(recon, dagger, kind, nthreads);
 }
+void launch_matpc_fused_f32(int recon, int dagger, const FusedArgs &f, int grid, cudaStream_t s) {
+    launch_matpc_fused_prec<4>(recon, dagger, f, grid, s);
+}
+int matpc_fused_wave_f32(int recon, int dagger) { return matpc_fused_wave<4>(recon, dagger); }
 }  // namespace qx

@@ -122,6 +122,22 @@ struct DslashArgs {
 };
 enum DslashRed { RED_NONE = 0, RED_XDOT_NORM = 1, RED_RHAT_DOT = 2 };
 
+// single-launch Mhat (matpc_fused.cuh): phase A = CLOVER_INV on odd, phase B = CLOVER_XPAY on even
+struct FusedArgs {
+    DslashArgs A, B;
+    int chunks;           // work items per timeslice and phase: ceil(F / threads)
+    int total_items;      // 2 T_loc chunks
+    const int *stages;    // [2 T_loc] dispense order: t (phase A) or T_loc + t (phase B)
+    unsigned *work;       // item counter, zero on entry
+    unsigned *doneA;      // [T_loc] completed phase-A chunks per timeslice, zero on entry
+};
+void launch_matpc_fused_f64(int recon, int dagger, const FusedArgs &f, int grid, cudaStream_t s);
+void launch_matpc_fused_f32(int recon, int dagger, const FusedArgs &f, int grid, cudaStream_t s);
+void launch_matpc_fused_f16(int recon, int dagger, const FusedArgs &f, int grid, cudaStream_t s);
+int matpc_fused_wave_f64(int recon, int dagger);
+int matpc_fused_wave_f32(int recon, int dagger);
+int matpc_fused_wave_f16(int recon, int dagger);
+
 void launch_dslash_f64(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
 void launch_dslash_f32(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
 void launch_dslash_f16(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
