@@ -147,7 +147,8 @@ static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int
         launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
         return;
     }
-    qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads, a.nrhs > 1 ? a.nrhs : 1};
+    qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads, a.nrhs > 1 ? a.nrhs : 1,
+                           a.red_kind};
     if (c->capturing) {  // graph: external event-record nodes, re-recorded at each replay
         QX_CUDA(cudaEventRecordWithFlags(r.a, c->stream, cudaEventRecordExternal));
         launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
@@ -172,6 +173,7 @@ static void rec_model(const qudax_ctx::TimingRec &r, qudax_site_model *out) {
     (void)hop;
     out->flops = m.flops * r.sites * r.nrhs;
     out->bytes_compulsory = ((m.bytes_compulsory - per_rhs) + per_rhs * r.nrhs) * r.sites;
+    if (r.red == RED_RHAT_DOT) out->bytes_compulsory += sp * r.sites;  // the fused <rhat0, out> reads rhat0
     out->bytes_paper = m.bytes_paper * r.sites * r.nrhs;
 }
 

@@ -33,6 +33,7 @@ struct qudax_ctx {
         int prec, recon, kind;
         long sites;
         int nrhs = 1;  // multi-RHS launch: links and clover are compulsory once, spinors per RHS
+        int red = 0;   // fused reduction kind (RED_RHAT_DOT reads rhat: +1 spinor per site)
     };
     std::vector<TimingRec> trecs;
     std::vector<cudaEvent_t> ev_pool;
