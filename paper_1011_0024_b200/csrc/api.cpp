@@ -238,14 +238,13 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     DslashArgs args = base_args(c, gc, prec, p, kind, a, reverse);
     args.in = in; args.out = out; args.x = x;
     int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
-    const int TPB = dslash_threads();
     const bool split = (c->comm == QUDAX_COMM_NCCL && c->overlap && g.T_loc > 2);
     const bool multi = (g.nranks > 1);  // cross-rank sums needed before the scalar recurrence
     if (red) {
         QX_CHECK(red->kind != RED_XDOT_NORM || kind == QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
         QX_CHECK(red->kind != RED_RHAT_DOT || red->rhat, QUDAX_ERR_ARG, "rhat-dot needs rhat");
         // CTA slots of up to two launches + their group slots (reduce.cuh)
-        if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / TPB) + 64)));
+        if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / 32) + 64)));
         args.red_kind = red->kind;
         args.rhat = red->rhat;
         const int ni = (int)((g.T_loc - 2) * g.F), nb = (int)(2 * g.F);
@@ -365,7 +364,7 @@ static void matpc_fused(qudax_ctx *c, void *out, const void *in, void *t, int pr
     if (red) {
         QX_CHECK(red->kind == RED_RHAT_DOT ? red->rhat != nullptr : red->kind == RED_XDOT_NORM, QUDAX_ERR_ARG,
                  "fused matpc: bad reduction");
-        if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / TPB) + 64)));
+        if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / 32) + 64)));
         f.B.red_kind = red->kind;
         f.B.rhat = red->rhat;
         f.B.tail.partials = c->dpart;

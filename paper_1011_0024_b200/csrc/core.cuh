@@ -31,6 +31,46 @@ template <typename R> __device__ __forceinline__ Cx<R> conj_mul(Cx<R> a, Cx<R> b
 template <typename R> __device__ __forceinline__ Cx<R> times_i(Cx<R> a) { return {-a.i, a.r}; }
 template <typename R> __device__ __forceinline__ R norm2(Cx<R> a) { return a.r * a.r + a.i * a.i; }
 
+// ---- fp32 complex arithmetic on the packed FP32x2 pipe (sm_100 FFMA2 / FADD2 / FMUL2).
+// A complex number is one register pair: an add or a real scale is one instruction instead of
+// two, and a complex multiply-accumulate two (scalar broadcast and pair-swap are operand
+// modifiers of FFMA2) instead of four.  These overloads take precedence over the templates
+// above for R = float; fp64 keeps the scalar forms.  Each lane rounds exactly as the scalar
+// FADD/FMUL/FFMA would; only the contraction pattern of complex products differs from the
+// compiler's scalar choice (within the fp32 / half parity tolerances).
+__device__ __forceinline__ float2 f2(Cx<float> a) { return make_float2(a.r, a.i); }
+__device__ __forceinline__ Cx<float> cf(float2 v) { return Cx<float>{v.x, v.y}; }
+__device__ __forceinline__ float2 bc(float s) { return make_float2(s, s); }
+__device__ __forceinline__ Cx<float> operator+(Cx<float> a, Cx<float> b) { return cf(__fadd2_rn(f2(a), f2(b))); }
+__device__ __forceinline__ Cx<float> operator-(Cx<float> a, Cx<float> b) {
+    return cf(__ffma2_rn(f2(b), bc(-1.f), f2(a)));
+}
+__device__ __forceinline__ Cx<float> operator*(float s, Cx<float> a) { return cf(__fmul2_rn(bc(s), f2(a))); }
+// i a as a pair: (-a.i, a.r)
+__device__ __forceinline__ float2 times_i2(Cx<float> a) { return __fmul2_rn(make_float2(a.i, a.r), make_float2(-1.f, 1.f)); }
+__device__ __forceinline__ Cx<float> operator*(Cx<float> a, Cx<float> b) {
+    return cf(__ffma2_rn(bc(a.i), times_i2(b), __fmul2_rn(bc(a.r), f2(b))));
+}
+__device__ __forceinline__ Cx<float> conj_mul(Cx<float> a, Cx<float> b) {
+    return cf(__ffma2_rn(bc(-a.i), times_i2(b), __fmul2_rn(bc(a.r), f2(b))));
+}
+
+// p + S i q (S = +-1): one FFMA2 in fp32 (pair swap as operand modifier)
+template <int S, typename R>
+__device__ __forceinline__ Cx<R> add_i(Cx<R> p, Cx<R> q) {
+    if constexpr (sizeof(R) == 4) {
+        return cf(__ffma2_rn(make_float2(q.i, q.r), make_float2((float)-S, (float)S), f2(p)));
+    } else {
+        return S > 0 ? Cx<R>{p.r - q.i, p.i + q.r} : Cx<R>{p.r + q.i, p.i - q.r};
+    }
+}
+// acc + s g (real s)
+template <typename R>
+__device__ __forceinline__ Cx<R> axpy(R s, Cx<R> g, Cx<R> acc) {
+    if constexpr (sizeof(R) == 4) return cf(__ffma2_rn(bc(s), f2(g), f2(acc)));
+    else return acc + s * g;
+}
+
 // ----------------------------------------------------------------------------- precision traits
 template <int P> struct Prec;
 template <> struct Prec<8> { using R = double; };
@@ -121,22 +161,34 @@ struct Blocks<4, NB, STREAM> {
 // ---- 16-bit fixed point <-> fp32 without the conversion (XU) pipe ------------------------
 // The paper's half precision relied on the GT200 texture unit to turn int16 into floats
 // (P:509-518).  On B200, I2F/F2I issue on the narrow XU pipe and become the limiter of the
-// half-precision Dslash (ncu: XU 60% busy).  Both directions are done with exact fp32
-// integer tricks on the ALU/FMA pipes instead:
-//   int16 s -> float: bits(0x4B000000 | (u16(s) ^ 0x8000)) = 2^23 + s + 2^15 exactly, minus
-//   (2^23 + 2^15);  float x (|x| <= 32767) -> RN-even int16: low 16 bits of bits(x + 1.5*2^23).
+// half-precision Dslash (ncu: XU 60% busy).  Both directions are exact fp32 integer tricks on
+// the ALU/FMA pipes instead.  A quantised value q in [-32767, 32767] is stored OFFSET-BINARY,
+// u = q + 32768 (the two's-complement bits with the sign bit flipped), so decoding is one
+// byte-permute per value: bits(0x4B000000 | u) = 2^23 + u exactly, minus (2^23 + 2^15) = q.
+//   float x (|x| <= 32767) -> RN-even u: low 16 bits of bits(x + 1.5*2^23 + 2^15).
+constexpr uint32_t kHalfMagic = 0x4B000000u;
+constexpr float kHalfBias = 8421376.0f;  // 2^23 + 2^15
 __device__ __forceinline__ float i16lo_to_f32(uint32_t w) {
-    return __uint_as_float((w & 0xFFFFu) ^ 0x4B008000u) - 8421376.0f;
+    return __uint_as_float(__byte_perm(w, kHalfMagic, 0x7610)) - kHalfBias;
 }
 __device__ __forceinline__ float i16hi_to_f32(uint32_t w) {
-    return __uint_as_float((w >> 16) ^ 0x4B008000u) - 8421376.0f;
+    return __uint_as_float(__byte_perm(w, kHalfMagic, 0x7632)) - kHalfBias;
 }
-// two already-scaled floats -> packed int16 pair (round to nearest even, as __float2int_rn)
+// both values of a stored word, times `scale`: 2 PRMT + FADD2 + FMUL2 (same rounding as the
+// scalar FADD then FMUL)
+__device__ __forceinline__ float2 dq2(uint32_t w, float scale) {
+    const float2 b = make_float2(__uint_as_float(__byte_perm(w, kHalfMagic, 0x7610)),
+                                 __uint_as_float(__byte_perm(w, kHalfMagic, 0x7632)));
+    return __fmul2_rn(bc(scale), __fadd2_rn(b, bc(-kHalfBias)));
+}
+// two already-scaled floats -> packed offset-binary pair (round to nearest even)
 __device__ __forceinline__ uint32_t f32x2_to_i16x2(float a, float b) {
-    const uint32_t ia = __float_as_uint(__fadd_rn(a, 12582912.0f));
-    const uint32_t ib = __float_as_uint(__fadd_rn(b, 12582912.0f));
+    const uint32_t ia = __float_as_uint(__fadd_rn(a, 12615680.0f));  // 1.5*2^23 + 2^15
+    const uint32_t ib = __float_as_uint(__fadd_rn(b, 12615680.0f));
     return __byte_perm(ia, ib, 0x5410);
 }
+// host/device: quantised integer q -> stored 16-bit word
+__host__ __device__ __forceinline__ short h16_code(int q) { return (short)(uint16_t)((unsigned)q ^ 0x8000u); }
 // the integer value held in a quantised word, as a float (exact)
 __device__ __forceinline__ float q_as_f32(float scaled) {
     return __uint_as_float(__float_as_uint(__fadd_rn(scaled, 12582912.0f))) - 12582912.0f;
@@ -157,10 +209,11 @@ struct Blocks<2, NB, STREAM> {
         for (int k = 0; k < NB; ++k) {
             uint2 v = STREAM == 1 ? ld_stream_u2(p + (b0 + k) * stride + i)
                       : (STREAM == 2 ? __ldcg(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i));
-            out[4 * k] = __fmul_rn(scale, i16lo_to_f32(v.x));
-            out[4 * k + 1] = __fmul_rn(scale, i16hi_to_f32(v.x));
-            out[4 * k + 2] = __fmul_rn(scale, i16lo_to_f32(v.y));
-            out[4 * k + 3] = __fmul_rn(scale, i16hi_to_f32(v.y));
+            const float2 a = dq2(v.x, scale), b = dq2(v.y, scale);
+            out[4 * k] = a.x;
+            out[4 * k + 1] = a.y;
+            out[4 * k + 2] = b.x;
+            out[4 * k + 3] = b.y;
         }
     }
     static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out) {
@@ -283,9 +336,9 @@ struct LinkIO {
             } else {
                 const short2 *p2 = reinterpret_cast<const short2 *>(reinterpret_cast<const char *>(base) +
                                                                     (size_t)NB4 * 8 * stride);
-                const uint32_t w = __ldg(reinterpret_cast<const uint32_t *>(p2) + i);
-                raw[RECON - 2] = __fmul_rn(kHalfInv, i16lo_to_f32(w));
-                raw[RECON - 1] = __fmul_rn(kHalfInv, i16hi_to_f32(w));
+                const float2 v = dq2(__ldg(reinterpret_cast<const uint32_t *>(p2) + i), kHalfInv);
+                raw[RECON - 2] = v.x;
+                raw[RECON - 1] = v.y;
             }
         }
     }
@@ -294,6 +347,9 @@ struct LinkIO {
     static __device__ __forceinline__ void load(const void *base, long stride, long i, Cx<R> u[3][3]) {
         R raw[RECON];
         load_raw(base, stride, i, raw);
+        reconstruct(raw, u);
+    }
+    static __device__ __forceinline__ void reconstruct(const R *raw, Cx<R> u[3][3]) {
         if constexpr (RECON == 18) {
 #pragma unroll
             for (int r = 0; r < 3; ++r)

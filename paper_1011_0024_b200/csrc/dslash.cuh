@@ -30,13 +30,49 @@ namespace qx {
 
 template <typename R>
 __device__ __forceinline__ void su3_mul(const Cx<R> u[3][3], const Cx<R> v[3], Cx<R> out[3]) {
+    if constexpr (sizeof(R) == 4) {  // 1 + 6 FFMA2 per row, i v shared by the rows
+        float2 iv[3];
 #pragma unroll
-    for (int a = 0; a < 3; ++a) out[a] = u[a][0] * v[0] + u[a][1] * v[1] + u[a][2] * v[2];
+        for (int c = 0; c < 3; ++c) iv[c] = times_i2(v[c]);
+#pragma unroll
+        for (int a = 0; a < 3; ++a) {
+            float2 acc = __fmul2_rn(bc(u[a][0].r), f2(v[0]));
+            acc = __ffma2_rn(bc(u[a][0].i), iv[0], acc);
+#pragma unroll
+            for (int c = 1; c < 3; ++c) {
+                acc = __ffma2_rn(bc(u[a][c].r), f2(v[c]), acc);
+                acc = __ffma2_rn(bc(u[a][c].i), iv[c], acc);
+            }
+            out[a] = cf(acc);
+        }
+    } else {
+#pragma unroll
+        for (int a = 0; a < 3; ++a) out[a] = u[a][0] * v[0] + u[a][1] * v[1] + u[a][2] * v[2];
+    }
 }
+// U^dag v: out[a] = sum_c conj(u[c][a]) v[c]
 template <typename R>
 __device__ __forceinline__ void su3_dag_mul(const Cx<R> u[3][3], const Cx<R> v[3], Cx<R> out[3]) {
+    if constexpr (sizeof(R) == 4) {
+        float2 iv[3];
 #pragma unroll
-    for (int a = 0; a < 3; ++a) out[a] = conj_mul(u[0][a], v[0]) + conj_mul(u[1][a], v[1]) + conj_mul(u[2][a], v[2]);
+        for (int c = 0; c < 3; ++c) iv[c] = times_i2(v[c]);
+#pragma unroll
+        for (int a = 0; a < 3; ++a) {
+            float2 acc = __fmul2_rn(bc(u[0][a].r), f2(v[0]));
+            acc = __ffma2_rn(bc(-u[0][a].i), iv[0], acc);
+#pragma unroll
+            for (int c = 1; c < 3; ++c) {
+                acc = __ffma2_rn(bc(u[c][a].r), f2(v[c]), acc);
+                acc = __ffma2_rn(bc(-u[c][a].i), iv[c], acc);
+            }
+            out[a] = cf(acc);
+        }
+    } else {
+#pragma unroll
+        for (int a = 0; a < 3; ++a)
+            out[a] = conj_mul(u[0][a], v[0]) + conj_mul(u[1][a], v[1]) + conj_mul(u[2][a], v[2]);
+    }
 }
 
 template <typename R>
@@ -48,22 +84,21 @@ __device__ __forceinline__ void unpack_spinor(const R *v, Cx<R> p[4][3]) {
 }
 
 // spatial hop: project psi with (1 + sigma gamma_mu), multiply by U (or U^dag), accumulate
+// (the projector formulas of the header, written with add_i(p, q) = p + S i q)
 template <int MU, int SIGMA, bool ADJ, typename R>
-__device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3][3], R coef, Cx<R> acc[4][3]) {
+__device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3][3], Cx<R> acc[4][3]) {
     Cx<R> h0[3], h1[3];
 #pragma unroll
     for (int c = 0; c < 3; ++c) {
-        if constexpr (MU == 0) {
-            Cx<R> a = times_i(p[3][c]), b = times_i(p[2][c]);
-            h0[c] = SIGMA > 0 ? p[0][c] - a : p[0][c] + a;
-            h1[c] = SIGMA > 0 ? p[1][c] - b : p[1][c] + b;
-        } else if constexpr (MU == 1) {
+        if constexpr (MU == 0) {  // h0 = p0 - s i p3, h1 = p1 - s i p2
+            h0[c] = add_i<-SIGMA>(p[0][c], p[3][c]);
+            h1[c] = add_i<-SIGMA>(p[1][c], p[2][c]);
+        } else if constexpr (MU == 1) {  // h0 = p0 + s p3, h1 = p1 - s p2
             h0[c] = SIGMA > 0 ? p[0][c] + p[3][c] : p[0][c] - p[3][c];
             h1[c] = SIGMA > 0 ? p[1][c] - p[2][c] : p[1][c] + p[2][c];
-        } else {
-            Cx<R> a = times_i(p[2][c]), b = times_i(p[3][c]);
-            h0[c] = SIGMA > 0 ? p[0][c] - a : p[0][c] + a;
-            h1[c] = SIGMA > 0 ? p[1][c] + b : p[1][c] - b;
+        } else {  // h0 = p0 - s i p2, h1 = p1 + s i p3
+            h0[c] = add_i<-SIGMA>(p[0][c], p[2][c]);
+            h1[c] = add_i<SIGMA>(p[1][c], p[3][c]);
         }
     }
     Cx<R> g0[3], g1[3];
@@ -76,21 +111,17 @@ __device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3
     }
 #pragma unroll
     for (int c = 0; c < 3; ++c) {
-        g0[c] = coef * g0[c];
-        g1[c] = coef * g1[c];
         acc[0][c] = acc[0][c] + g0[c];
         acc[1][c] = acc[1][c] + g1[c];
-        if constexpr (MU == 0) {
-            Cx<R> a = times_i(g1[c]), b = times_i(g0[c]);
-            acc[2][c] = SIGMA > 0 ? acc[2][c] + a : acc[2][c] - a;
-            acc[3][c] = SIGMA > 0 ? acc[3][c] + b : acc[3][c] - b;
-        } else if constexpr (MU == 1) {
+        if constexpr (MU == 0) {  // r2 = s i h1, r3 = s i h0
+            acc[2][c] = add_i<SIGMA>(acc[2][c], g1[c]);
+            acc[3][c] = add_i<SIGMA>(acc[3][c], g0[c]);
+        } else if constexpr (MU == 1) {  // r2 = -s h1, r3 = s h0
             acc[2][c] = SIGMA > 0 ? acc[2][c] - g1[c] : acc[2][c] + g1[c];
             acc[3][c] = SIGMA > 0 ? acc[3][c] + g0[c] : acc[3][c] - g0[c];
-        } else {
-            Cx<R> a = times_i(g0[c]), b = times_i(g1[c]);
-            acc[2][c] = SIGMA > 0 ? acc[2][c] + a : acc[2][c] - a;
-            acc[3][c] = SIGMA > 0 ? acc[3][c] - b : acc[3][c] + b;
+        } else {  // r2 = s i h0, r3 = -s i h1
+            acc[2][c] = add_i<SIGMA>(acc[2][c], g0[c]);
+            acc[3][c] = add_i<-SIGMA>(acc[3][c], g1[c]);
         }
     }
 }
@@ -114,25 +145,47 @@ __device__ __forceinline__ void temporal_hop(const R *hv, const Cx<R> u[3][3], R
     constexpr int s0 = UPPER ? 0 : 2;
 #pragma unroll
     for (int c = 0; c < 3; ++c) {
-        acc[s0][c] = acc[s0][c] + coef * g0[c];
-        acc[s0 + 1][c] = acc[s0 + 1][c] + coef * g1[c];
+        acc[s0][c] = axpy(coef, g0[c], acc[s0][c]);
+        acc[s0 + 1][c] = axpy(coef, g1[c], acc[s0 + 1][c]);
     }
 }
 
 // Hermitian 6x6 (d[6], lower triangle L[15]) times v
 template <typename R>
 __device__ __forceinline__ void herm6_mul(const R *m, const Cx<R> v[6], Cx<R> out[6]) {
+    if constexpr (sizeof(R) == 4) {  // out_i += L v_j and out_j += conj(L) v_i: 2 FFMA2 each
+        float2 iv[6], o[6];
 #pragma unroll
-    for (int i = 0; i < 6; ++i) out[i] = m[i] * v[i];
-#pragma unroll
-    for (int i = 1; i < 6; ++i)
-#pragma unroll
-        for (int j = 0; j < i; ++j) {
-            const int k = i * (i - 1) / 2 + j;
-            Cx<R> L = cx(m[6 + 2 * k], m[6 + 2 * k + 1]);
-            out[i] = out[i] + L * v[j];
-            out[j] = out[j] + conj_mul(L, v[i]);
+        for (int i = 0; i < 6; ++i) {
+            iv[i] = times_i2(v[i]);
+            o[i] = __fmul2_rn(bc(m[i]), f2(v[i]));
         }
+#pragma unroll
+        for (int i = 1; i < 6; ++i)
+#pragma unroll
+            for (int j = 0; j < i; ++j) {
+                const int k = i * (i - 1) / 2 + j;
+                const float Lr = m[6 + 2 * k], Li = m[6 + 2 * k + 1];
+                o[i] = __ffma2_rn(bc(Lr), f2(v[j]), o[i]);
+                o[i] = __ffma2_rn(bc(Li), iv[j], o[i]);
+                o[j] = __ffma2_rn(bc(Lr), f2(v[i]), o[j]);
+                o[j] = __ffma2_rn(bc(-Li), iv[i], o[j]);
+            }
+#pragma unroll
+        for (int i = 0; i < 6; ++i) out[i] = cf(o[i]);
+    } else {
+#pragma unroll
+        for (int i = 0; i < 6; ++i) out[i] = m[i] * v[i];
+#pragma unroll
+        for (int i = 1; i < 6; ++i)
+#pragma unroll
+            for (int j = 0; j < i; ++j) {
+                const int k = i * (i - 1) / 2 + j;
+                Cx<R> L = cx(m[6 + 2 * k], m[6 + 2 * k + 1]);
+                out[i] = out[i] + L * v[j];
+                out[j] = out[j] + conj_mul(L, v[i]);
+            }
+    }
 }
 
 template <int P>
@@ -188,10 +241,10 @@ __device__ __forceinline__ void apply_clover(const void *cl, long stride, long i
 #define QX_DSLASH_THREADS 128
 #endif
 // Minimum resident CTAs per SM (register cap).  Measured on B200 at 32^3x64
-// (profiles/r01_variants.log): fp32 needs >= 7 x 128 threads in flight per SM to cover HBM
-// latency (72 regs, small L1-resident spills), fp64 must not be capped (152 regs; capping
-// spills and loses 20%).
-template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) ? 1 : 7; };
+// (profiles/r01_variants.log): fp32 / half need >= 6 x 128 threads in flight per SM to cover
+// HBM latency (80 regs; with the packed FP32x2 math 7 x 128 = 72 regs spilled more and lost
+// 3-8%), fp64 must not be capped (152 regs; capping spills and loses 20%).
+template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) ? 1 : 6; };
 #ifdef QX_DSLASH_MINB
 #define QX_MINB_OF(P) QX_DSLASH_MINB
 #else
@@ -258,11 +311,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[0][p], a.stride, i, u);
-        spatial_hop<0, SF, false>(ps, u, (R)1, acc);
+        spatial_hop<0, SF, false>(ps, u, acc);
         SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[0][op], a.stride, nb, u);
-        spatial_hop<0, SB, true>(ps, u, (R)1, acc);
+        spatial_hop<0, SB, true>(ps, u, acc);
     }
     // ---- y direction
     {
@@ -273,11 +326,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[1][p], a.stride, i, u);
-        spatial_hop<1, SF, false>(ps, u, (R)1, acc);
+        spatial_hop<1, SF, false>(ps, u, acc);
         SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[1][op], a.stride, nb, u);
-        spatial_hop<1, SB, true>(ps, u, (R)1, acc);
+        spatial_hop<1, SB, true>(ps, u, acc);
     }
     // ---- z direction
     {
@@ -288,11 +341,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[2][p], a.stride, i, u);
-        spatial_hop<2, SF, false>(ps, u, (R)1, acc);
+        spatial_hop<2, SF, false>(ps, u, acc);
         SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
         unpack_spinor(v, ps);
         LinkIO<P, RECON>::load(a.gauge[2][op], a.stride, nb, u);
-        spatial_hop<2, SB, true>(ps, u, (R)1, acc);
+        spatial_hop<2, SB, true>(ps, u, acc);
     }
     // ---- t direction: diagonal projectors, 12 reals per neighbour (eq. (6))
     {

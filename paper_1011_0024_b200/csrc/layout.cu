@@ -158,7 +158,7 @@ __device__ void encode_store_link(const double *l /*18*/, void *base, long strid
     } else {
         short4 *p = reinterpret_cast<short4 *>(base);
         constexpr int NB = RECON / 4;
-        auto q16 = [](double v) { return (short)__double2int_rn(v * 32767.0); };
+        auto q16 = [](double v) { return h16_code(__double2int_rn(v * 32767.0)); };
         for (int k = 0; k < NB; ++k) {
             short4 v;
             v.x = q16(raw[4 * k]); v.y = q16(raw[4 * k + 1]); v.z = q16(raw[4 * k + 2]); v.w = q16(raw[4 * k + 3]);
@@ -415,10 +415,10 @@ __global__ void k_clover_pack(long Vh, long stride, const double *__restrict__ s
             const float inv = m > 0 ? kHalfMax / (float)m : 0.f;
             for (int k = 0; k < 9; ++k) {
                 short4 v;
-                v.x = (short)__float2int_rn((float)s[36 * b + 4 * k] * inv);
-                v.y = (short)__float2int_rn((float)s[36 * b + 4 * k + 1] * inv);
-                v.z = (short)__float2int_rn((float)s[36 * b + 4 * k + 2] * inv);
-                v.w = (short)__float2int_rn((float)s[36 * b + 4 * k + 3] * inv);
+                v.x = h16_code(__float2int_rn((float)s[36 * b + 4 * k] * inv));
+                v.y = h16_code(__float2int_rn((float)s[36 * b + 4 * k + 1] * inv));
+                v.z = h16_code(__float2int_rn((float)s[36 * b + 4 * k + 2] * inv));
+                v.w = h16_code(__float2int_rn((float)s[36 * b + 4 * k + 3] * inv));
                 p[(9 * b + k) * stride + i] = v;
             }
         }
