@@ -4,6 +4,7 @@
 #pragma once
 #include <cuda_runtime.h>
 #include <cstdint>
+#include <type_traits>
 
 namespace qx {
 
@@ -401,6 +402,107 @@ struct LinkIO {
     static __device__ __forceinline__ float sqrt_(float x) { return x * rsqrtf(fmaxf(x, 1e-30f)); }
     static __device__ __forceinline__ double rcp_(double x) { return 1.0 / x; }
     static __device__ __forceinline__ float rcp_(float x) { return __fdividef(1.0f, x); }
+};
+
+// ----------------------------------------------------------------------------- raw site data
+// Undecoded loads, so the Dslash can issue the loads of two hops before consuming either
+// (half: the 16-bit words + norm stay packed, half the registers of the decoded values).
+template <int P> struct StoreVec;
+template <> struct StoreVec<8> { using V = double2; };
+template <> struct StoreVec<4> { using V = float4; };
+template <> struct StoreVec<2> { using V = uint2; };
+
+template <int P, int NB>
+struct RawVec {
+    using V = typename StoreVec<P>::V;
+    using R = typename Prec<P>::R;
+    V d[NB];
+    float n;  // half: the site norm
+    // blocks [b0, b0 + NB) of site i; `norms` = the norm array (half only)
+    template <int MODE>
+    __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, const float *norms) {
+        const V *p = reinterpret_cast<const V *>(base);
+#pragma unroll
+        for (int k = 0; k < NB; ++k) d[k] = MODE == 2 ? __ldcg(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
+        if constexpr (P == 2) n = MODE == 2 ? __ldcg(norms + i) : __ldg(norms + i);
+    }
+    // identical values to SpinorIO / FaceIO loads
+    __device__ __forceinline__ void decode(R *out) const {
+        if constexpr (P == 8) {
+#pragma unroll
+            for (int k = 0; k < NB; ++k) {
+                out[2 * k] = d[k].x;
+                out[2 * k + 1] = d[k].y;
+            }
+        } else if constexpr (P == 4) {
+#pragma unroll
+            for (int k = 0; k < NB; ++k) {
+                out[4 * k] = d[k].x; out[4 * k + 1] = d[k].y; out[4 * k + 2] = d[k].z; out[4 * k + 3] = d[k].w;
+            }
+        } else {
+            const float scale = n * kHalfInv;
+#pragma unroll
+            for (int k = 0; k < NB; ++k) {
+                const float2 a = dq2(d[k].x, scale), b = dq2(d[k].y, scale);
+                out[4 * k] = a.x; out[4 * k + 1] = a.y; out[4 * k + 2] = b.x; out[4 * k + 3] = b.y;
+            }
+        }
+    }
+};
+
+template <int P, int RECON>
+struct RawLink {
+    using V = typename StoreVec<P>::V;
+    using R = typename Prec<P>::R;
+    static constexpr int NB = (P == 8) ? RECON / 2 : RECON / 4;
+    static constexpr bool kTail = (P != 8) && (RECON % 4) != 0;
+    V d[NB];
+    typename std::conditional<P == 4, float2, uint32_t>::type tail;
+    __device__ __forceinline__ void load(const void *base, long stride, long i) {
+        const V *p = reinterpret_cast<const V *>(base);
+#pragma unroll
+        for (int k = 0; k < NB; ++k) {
+            if constexpr (P == 2) d[k] = ld_stream_u2(p + k * stride + i);
+            else d[k] = ld_stream(p + k * stride + i);
+        }
+        if constexpr (kTail) {
+            const char *t = reinterpret_cast<const char *>(base) + (size_t)NB * sizeof(V) * stride;
+            if constexpr (P == 4) tail = ld_stream(reinterpret_cast<const float2 *>(t) + i);
+            else tail = __ldg(reinterpret_cast<const uint32_t *>(t) + i);
+        }
+    }
+    // identical to LinkIO<P, RECON>::load
+    __device__ __forceinline__ void decode(Cx<R> u[3][3]) const {
+        R raw[RECON];
+        if constexpr (P == 8) {
+#pragma unroll
+            for (int k = 0; k < NB; ++k) {
+                raw[2 * k] = d[k].x;
+                raw[2 * k + 1] = d[k].y;
+            }
+        } else if constexpr (P == 4) {
+#pragma unroll
+            for (int k = 0; k < NB; ++k) {
+                raw[4 * k] = d[k].x; raw[4 * k + 1] = d[k].y; raw[4 * k + 2] = d[k].z; raw[4 * k + 3] = d[k].w;
+            }
+            if constexpr (kTail) {
+                raw[RECON - 2] = tail.x;
+                raw[RECON - 1] = tail.y;
+            }
+        } else {
+#pragma unroll
+            for (int k = 0; k < NB; ++k) {
+                const float2 a = dq2(d[k].x, kHalfInv), b = dq2(d[k].y, kHalfInv);
+                raw[4 * k] = a.x; raw[4 * k + 1] = a.y; raw[4 * k + 2] = b.x; raw[4 * k + 3] = b.y;
+            }
+            if constexpr (kTail) {
+                const float2 v = dq2(tail, kHalfInv);
+                raw[RECON - 2] = v.x;
+                raw[RECON - 1] = v.y;
+            }
+        }
+        LinkIO<P, RECON>::reconstruct(raw, u);
+    }
 };
 
 }  // namespace qx

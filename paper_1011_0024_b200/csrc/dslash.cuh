@@ -237,6 +237,17 @@ __device__ __forceinline__ void apply_clover(const void *cl, long stride, long i
         }
 }
 
+// Whether a direction issues both hops' loads before computing either (measured,
+// profiles/r01_variants.log): fp64 yes (+4%), fp32 no (spills at the 80-register cap), half
+// yes except recon-12 (within 3%).  QX_PAIR_MASK overrides: bit 0 half, 1 fp32, 2 fp64.
+template <int P, int RECON>
+__host__ __device__ constexpr bool dslash_pair() {
+#ifdef QX_PAIR_MASK
+    return (QX_PAIR_MASK >> (P == 2 ? 0 : (P == 4 ? 1 : 2))) & 1;
+#else
+    return P == 8 || (P == 2 && RECON != 12);
+#endif
+}
 #ifndef QX_DSLASH_THREADS
 #define QX_DSLASH_THREADS 128
 #endif
@@ -302,91 +313,98 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     constexpr int SF = DAG ? +1 : -1;  // sigma of the forward hop
     constexpr int SB = -SF;
 
-    // ---- x direction
-    {
-        const int nf = (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1;
-        const int nb = (x == 0 ? lex + (X - 1) : lex - 1) >> 1;
-        R v[24];
-        Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
-        unpack_spinor(v, ps);
-        LinkIO<P, RECON>::load(a.gauge[0][p], a.stride, i, u);
-        spatial_hop<0, SF, false>(ps, u, acc);
-        SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
-        unpack_spinor(v, ps);
-        LinkIO<P, RECON>::load(a.gauge[0][op], a.stride, nb, u);
-        spatial_hop<0, SB, true>(ps, u, acc);
-    }
-    // ---- y direction
-    {
-        const int nf = (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1;
-        const int nb = (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1;
-        R v[24];
-        Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
-        unpack_spinor(v, ps);
-        LinkIO<P, RECON>::load(a.gauge[1][p], a.stride, i, u);
-        spatial_hop<1, SF, false>(ps, u, acc);
-        SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
-        unpack_spinor(v, ps);
-        LinkIO<P, RECON>::load(a.gauge[1][op], a.stride, nb, u);
-        spatial_hop<1, SB, true>(ps, u, acc);
-    }
-    // ---- z direction
-    {
-        const int nf = (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1;
-        const int nb = (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1;
-        R v[24];
-        Cx<R> ps[4][3], u[3][3];
-        SpinorIO<P>::template load<INMODE>(fin,a.stride, nf, v);
-        unpack_spinor(v, ps);
-        LinkIO<P, RECON>::load(a.gauge[2][p], a.stride, i, u);
-        spatial_hop<2, SF, false>(ps, u, acc);
-        SpinorIO<P>::template load<INMODE>(fin,a.stride, nb, v);
-        unpack_spinor(v, ps);
-        LinkIO<P, RECON>::load(a.gauge[2][op], a.stride, nb, u);
-        spatial_hop<2, SB, true>(ps, u, acc);
-    }
+    // Each direction loads raw (undecoded) neighbour spinors and links.  With PAIR the loads
+    // of the backward hop are issued before the forward hop is computed: twice the bytes in
+    // flight per thread (dslash_pair).
+    constexpr bool PAIR = dslash_pair<P, RECON>();
+    constexpr int NBS = (P == 8) ? 12 : 6;  // storage blocks of a spinor
+    const float *nrm = SpinorIO<P>::norms(fin, a.stride);
+    auto spatial = [&](auto mu_c, int nf, int nb) {
+        constexpr int MU = decltype(mu_c)::value;
+        RawVec<P, NBS> sf, sb;
+        RawLink<P, RECON> lf, lb;
+        sf.template load<INMODE>(fin, a.stride, nf, 0, nrm);
+        lf.load(a.gauge[MU][p], a.stride, i);
+        if constexpr (PAIR) {
+            sb.template load<INMODE>(fin, a.stride, nb, 0, nrm);
+            lb.load(a.gauge[MU][op], a.stride, nb);
+        }
+        {
+            R v[24];
+            Cx<R> ps[4][3], u[3][3];
+            sf.decode(v);
+            unpack_spinor(v, ps);
+            lf.decode(u);
+            spatial_hop<MU, SF, false>(ps, u, acc);
+        }
+        if constexpr (!PAIR) {
+            sb.template load<INMODE>(fin, a.stride, nb, 0, nrm);
+            lb.load(a.gauge[MU][op], a.stride, nb);
+        }
+        {
+            R v[24];
+            Cx<R> ps[4][3], u[3][3];
+            sb.decode(v);
+            unpack_spinor(v, ps);
+            lb.decode(u);
+            spatial_hop<MU, SB, true>(ps, u, acc);
+        }
+    };
+    spatial(std::integral_constant<int, 0>{}, (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1,
+            (x == 0 ? lex + (X - 1) : lex - 1) >> 1);
+    spatial(std::integral_constant<int, 1>{}, (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1,
+            (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1);
+    spatial(std::integral_constant<int, 2>{}, (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1,
+            (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1);
+
     // ---- t direction: diagonal projectors, 12 reals per neighbour (eq. (6))
     {
-        // forward: (1 + SF gamma_4): SF = -1 -> lower spins, SF = +1 -> upper spins
-        constexpr bool FWD_UPPER = (SF > 0);
-        const int T_loc = a.T_loc;
-        R h[12];
-        Cx<R> u[3][3];
-        R cf = (R)2;
-        if (t == T_loc - 1) {
-            cf = (R)(2.0 * a.bc_fwd);
-            if (a.ghosted) {
-                FaceIO<P>::load(a.ghost_fwd, a.fstride, i - t * a.F, h);
-            } else {
-                SpinorIO<P>::template load_half<INMODE>(fin,a.stride, (lex - (T_loc - 1) * XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
-            }
-        } else {
-            SpinorIO<P>::template load_half<INMODE>(fin,a.stride, (lex + XYZ) >> 1, FWD_UPPER ? 0 : 1, h);
-        }
-        LinkIO<P, RECON>::load(a.gauge[3][p], a.stride, i, u);
-        temporal_hop<FWD_UPPER, false>(h, u, cf, acc);
-
+        // forward: (1 + SF gamma_4): SF = -1 -> lower spins, SF = +1 -> upper spins;
         // backward: (1 + SB gamma_4)
+        constexpr bool FWD_UPPER = (SF > 0);
         constexpr bool BWD_UPPER = (SB > 0);
-        R cb = (R)2;
-        if (t == 0) {
-            cb = (R)(2.0 * a.bc_back);
-            if (a.ghosted) {
-                FaceIO<P>::load(a.ghost_back, a.fstride, i, h);
-                LinkIO<P, RECON>::load(a.gauge_ghost, a.fstride, i, u);
+        constexpr int NBH = NBS / 2;
+        const int T_loc = a.T_loc;
+        // operand addresses first (ghost face / periodic wrap / interior), then one load each
+        const bool fwd_ghost = (t == T_loc - 1) && a.ghosted;
+        const bool bwd_ghost = (t == 0) && a.ghosted;
+        const R cf = (t == T_loc - 1) ? (R)(2.0 * a.bc_fwd) : (R)2;
+        const R cb = (t == 0) ? (R)(2.0 * a.bc_back) : (R)2;
+        const int nfw = (t == T_loc - 1 ? lex - (T_loc - 1) * XYZ : lex + XYZ) >> 1;
+        const int nbw = (t == 0 ? lex + (T_loc - 1) * XYZ : lex - XYZ) >> 1;
+        RawVec<P, NBH> hf, hb;
+        RawLink<P, RECON> lf, lb;
+        auto load_f = [&] {
+            if (fwd_ghost) hf.template load<0>(a.ghost_fwd, a.fstride, i - t * a.F, 0, FaceIO<P>::norms(a.ghost_fwd, a.fstride));
+            else hf.template load<INMODE>(fin, a.stride, nfw, FWD_UPPER ? 0 : NBH, nrm);
+            lf.load(a.gauge[3][p], a.stride, i);
+        };
+        auto load_b = [&] {
+            if (bwd_ghost) {
+                hb.template load<0>(a.ghost_back, a.fstride, i, 0, FaceIO<P>::norms(a.ghost_back, a.fstride));
+                lb.load(a.gauge_ghost, a.fstride, i);
             } else {
-                const int nb = (lex + (T_loc - 1) * XYZ) >> 1;
-                SpinorIO<P>::template load_half<INMODE>(fin,a.stride, nb, BWD_UPPER ? 0 : 1, h);
-                LinkIO<P, RECON>::load(a.gauge[3][op], a.stride, nb, u);
+                hb.template load<INMODE>(fin, a.stride, nbw, BWD_UPPER ? 0 : NBH, nrm);
+                lb.load(a.gauge[3][op], a.stride, nbw);
             }
-        } else {
-            const int nb = (lex - XYZ) >> 1;
-            SpinorIO<P>::template load_half<INMODE>(fin,a.stride, nb, BWD_UPPER ? 0 : 1, h);
-            LinkIO<P, RECON>::load(a.gauge[3][op], a.stride, nb, u);
+        };
+        load_f();
+        if constexpr (PAIR) load_b();
+        {
+            R h[12];
+            Cx<R> u[3][3];
+            hf.decode(h);
+            lf.decode(u);
+            temporal_hop<FWD_UPPER, false>(h, u, cf, acc);
         }
-        temporal_hop<BWD_UPPER, true>(h, u, cb, acc);
+        if constexpr (!PAIR) load_b();
+        {
+            R h[12];
+            Cx<R> u[3][3];
+            hb.decode(h);
+            lb.decode(u);
+            temporal_hop<BWD_UPPER, true>(h, u, cb, acc);
+        }
     }
 
     // ---- epilogue: fused clover
