@@ -200,49 +200,73 @@ __device__ __forceinline__ uint2 ld_stream_u2(const uint2 *p) {
     return v;
 }
 
-// half: raw integer values scaled by `scale` (norm/32767 for spinors, 1/32767 for links)
-template <int NB, int STREAM>
-struct Blocks<2, NB, STREAM> {
-    static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out,
-                                                float scale) {
-        const uint2 *p = reinterpret_cast<const uint2 *>(base);
+
+// ---- half storage records.  Every 16-bit field is stored in 16-byte words first: a 12-real
+// record (half spinor, face, recon-12 link) is one uint4 (reals 0-7) + one uint2 (reals 8-11),
+// each in its own site-major region, so a warp load moves 512 B per instruction (an 8-byte
+// layout needs twice the load instructions and outstanding requests per byte).
+__device__ __forceinline__ uint4 ld_stream_u4(const uint4 *p) {
+    uint4 v;
+    asm volatile("ld.global.nc.L1::no_allocate.v4.u32 {%0,%1,%2,%3}, [%4];"
+                 : "=r"(v.x), "=r"(v.y), "=r"(v.z), "=r"(v.w) : "l"(p));
+    return v;
+}
+// MODE 0: read-only path; 1: streamed (no L1 allocation); 2: L2 only (coherent)
+template <int MODE, typename V>
+__device__ __forceinline__ V ld_m(const V *p) {
+    if constexpr (MODE == 2) return __ldcg(p);
+    else if constexpr (MODE == 1) {
+        if constexpr (std::is_same<V, uint4>::value) return ld_stream_u4(p);
+        else if constexpr (std::is_same<V, uint2>::value) return ld_stream_u2(p);
+        else return __ldg(p);
+    } else return __ldg(p);
+}
+struct H12 {
+    uint4 u;
+    uint2 v;
+    template <int MODE>
+    __device__ __forceinline__ void load(const void *ureg, const void *vreg, long i) {
+        u = ld_m<MODE>(reinterpret_cast<const uint4 *>(ureg) + i);
+        v = ld_m<MODE>(reinterpret_cast<const uint2 *>(vreg) + i);
+    }
+    __device__ __forceinline__ void decode(float scale, float *out) const {
+        const uint32_t w[6] = {u.x, u.y, u.z, u.w, v.x, v.y};
 #pragma unroll
-        for (int k = 0; k < NB; ++k) {
-            uint2 v = STREAM == 1 ? ld_stream_u2(p + (b0 + k) * stride + i)
-                      : (STREAM == 2 ? __ldcg(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i));
-            const float2 a = dq2(v.x, scale), b = dq2(v.y, scale);
-            out[4 * k] = a.x;
-            out[4 * k + 1] = a.y;
-            out[4 * k + 2] = b.x;
-            out[4 * k + 3] = b.y;
+        for (int k = 0; k < 6; ++k) {
+            const float2 d = dq2(w[k], scale);
+            out[2 * k] = d.x;
+            out[2 * k + 1] = d.y;
         }
     }
-    static __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, float *out) {
-        load(base, stride, i, b0, out, kHalfInv);
-    }
-    // quantise (value * inv_scale, round to nearest even) and store
-    static __device__ __forceinline__ void store_q(void *base, long stride, long i, int b0, const float *in,
-                                                   float inv_scale) {
-        uint2 *p = reinterpret_cast<uint2 *>(base);
+    __device__ __forceinline__ void encode(const float *in, float inv) {
+        uint32_t w[6];
 #pragma unroll
-        for (int k = 0; k < NB; ++k) {
-            uint2 v;
-            v.x = f32x2_to_i16x2(__fmul_rn(in[4 * k], inv_scale), __fmul_rn(in[4 * k + 1], inv_scale));
-            v.y = f32x2_to_i16x2(__fmul_rn(in[4 * k + 2], inv_scale), __fmul_rn(in[4 * k + 3], inv_scale));
-            p[(b0 + k) * stride + i] = v;
-        }
+        for (int k = 0; k < 6; ++k) w[k] = f32x2_to_i16x2(__fmul_rn(in[2 * k], inv), __fmul_rn(in[2 * k + 1], inv));
+        u = make_uint4(w[0], w[1], w[2], w[3]);
+        v = make_uint2(w[4], w[5]);
+    }
+    __device__ __forceinline__ void store(void *ureg, void *vreg, long i) const {
+        reinterpret_cast<uint4 *>(ureg)[i] = u;
+        reinterpret_cast<uint2 *>(vreg)[i] = v;
     }
 };
+// region addresses.  Half spinor field: [U upper][U lower][V upper][V lower][norm] x stride;
+// face: [U][V][norm] x fstride.
+__device__ __forceinline__ const char *cptr(const void *b, size_t off) { return reinterpret_cast<const char *>(b) + off; }
+__device__ __forceinline__ char *mptr(void *b, size_t off) { return reinterpret_cast<char *>(b) + off; }
+__device__ __forceinline__ size_t h_spinor_u(long stride, int hf) { return (size_t)16 * stride * hf; }
+__device__ __forceinline__ size_t h_spinor_v(long stride, int hf) { return (size_t)(32 + 8 * hf) * stride; }
 
 // ----------------------------------------------------------------------------- spinors
 // A spinor field: 24 reals per site (spin-major, colour, re/im) in the NR basis.
-// fp64: 12 double2 blocks; fp32: 6 float4 blocks; half: 6 short4 blocks + float norm[stride].
+// fp64: 12 double2 blocks; fp32: 6 float4 blocks; half: two H12 records (upper spins 0,1 and
+// lower spins 2,3) + float norm[stride].
 template <int P>
 struct SpinorIO {
     using R = typename Prec<P>::R;
     static constexpr int BPH = (P == 8) ? 6 : 3;  // blocks per 12-real half-spinor
 
-    // norm array (half only) follows the 6 short4 blocks
+    // norm array (half only) follows the 48 bytes x stride of the four half regions
     static __device__ __forceinline__ const float *norms(const void *base, long stride) {
         return reinterpret_cast<const float *>(reinterpret_cast<const char *>(base) + (size_t)6 * 8 * stride);
     }
@@ -255,8 +279,10 @@ struct SpinorIO {
     template <int MODE = 0>
     static __device__ __forceinline__ void load_half(const void *base, long stride, long i, int half, R *out) {
         if constexpr (P == 2) {
-            float nrm = MODE == 2 ? __ldcg(norms(base, stride) + i) : __ldg(norms(base, stride) + i);
-            Blocks<2, 3, MODE>::load(base, stride, i, 3 * half, out, nrm * kHalfInv);
+            const float nrm = ld_m<MODE>(norms(base, stride) + i);
+            H12 r;
+            r.load<MODE>(cptr(base, h_spinor_u(stride, half)), cptr(base, h_spinor_v(stride, half)), i);
+            r.decode(nrm * kHalfInv, out);
         } else {
             Blocks<P, BPH, MODE>::load(base, stride, i, BPH * half, out);
         }
@@ -272,8 +298,13 @@ struct SpinorIO {
 #pragma unroll
             for (int k = 0; k < 24; ++k) m = fmaxf(m, fabsf(in[k]));
             norms(base, stride)[i] = m;
-            float inv = (m > 0.f) ? kHalfMax / m : 0.f;
-            Blocks<2, 6, false>::store_q(base, stride, i, 0, in, inv);
+            const float inv = (m > 0.f) ? kHalfMax / m : 0.f;
+#pragma unroll
+            for (int hf = 0; hf < 2; ++hf) {
+                H12 r;
+                r.encode(in + 12 * hf, inv);
+                r.store(mptr(base, h_spinor_u(stride, hf)), mptr(base, h_spinor_v(stride, hf)), i);
+            }
         } else {
             Blocks<P, 2 * BPH, false>::store(base, stride, i, 0, in);
         }
@@ -295,7 +326,7 @@ struct SpinorIO {
     }
 };
 
-// A face (12 reals per site): fp64 6 double2, fp32 3 float4, half 3 short4 + float norm[fstride]
+// A face (12 reals per site): fp64 6 double2, fp32 3 float4, half one H12 + float norm[fstride]
 template <int P>
 struct FaceIO {
     using R = typename Prec<P>::R;
@@ -308,10 +339,55 @@ struct FaceIO {
     }
     static __device__ __forceinline__ void load(const void *base, long fs, long f, R *out) {
         if constexpr (P == 2) {
-            float nrm = __ldg(norms(base, fs) + f);
-            Blocks<2, 3, false>::load(base, fs, f, 0, out, nrm * kHalfInv);
+            const float nrm = __ldg(norms(base, fs) + f);
+            H12 r;
+            r.load<0>(base, cptr(base, (size_t)16 * fs), f);
+            r.decode(nrm * kHalfInv, out);
         } else {
             Blocks<P, NB, false>::load(base, fs, f, 0, out);
+        }
+    }
+};
+
+// Half links: RECON/8 uint4 regions, then a uint2 region (RECON % 8 == 4), then a uint32
+// region (RECON % 4 == 2) — recon-12: 16 + 8 B, recon-18: 16 + 16 + 4 B, recon-8: 16 B.
+template <int RECON>
+struct HLink {
+    static constexpr int N16 = RECON / 8;
+    static constexpr bool kV = (RECON % 8) >= 4;
+    static constexpr bool kW = (RECON % 4) == 2;
+    uint4 u[N16];
+    uint2 v;
+    uint32_t w;
+    __device__ __forceinline__ void load(const void *base, long stride, long i) {
+#pragma unroll
+        for (int k = 0; k < N16; ++k) u[k] = ld_stream_u4(reinterpret_cast<const uint4 *>(cptr(base, (size_t)16 * k * stride)) + i);
+        size_t off = (size_t)16 * N16 * stride;
+        if constexpr (kV) {
+            v = ld_stream_u2(reinterpret_cast<const uint2 *>(cptr(base, off)) + i);
+            off += (size_t)8 * stride;
+        }
+        if constexpr (kW) w = __ldg(reinterpret_cast<const uint32_t *>(cptr(base, off)) + i);
+    }
+    __device__ __forceinline__ void decode(float *raw) const {
+#pragma unroll
+        for (int k = 0; k < N16; ++k) {
+            const uint32_t q[4] = {u[k].x, u[k].y, u[k].z, u[k].w};
+#pragma unroll
+            for (int j = 0; j < 4; ++j) {
+                const float2 d = dq2(q[j], kHalfInv);
+                raw[8 * k + 2 * j] = d.x;
+                raw[8 * k + 2 * j + 1] = d.y;
+            }
+        }
+        if constexpr (kV) {
+            const float2 a = dq2(v.x, kHalfInv), b = dq2(v.y, kHalfInv);
+            raw[8 * N16] = a.x; raw[8 * N16 + 1] = a.y; raw[8 * N16 + 2] = b.x; raw[8 * N16 + 3] = b.y;
+        }
+        if constexpr (kW) {
+            const float2 a = dq2(w, kHalfInv);
+            raw[RECON - 2] = a.x;
+            raw[RECON - 1] = a.y;
         }
     }
 };
@@ -324,20 +400,17 @@ template <int P, int RECON>
 struct LinkIO {
     using R = typename Prec<P>::R;
     static __device__ __forceinline__ void load_raw(const void *base, long stride, long i, R *raw) {
-        constexpr int NB4 = (P == 8) ? RECON / 2 : RECON / 4;
-        Blocks<P, NB4, true>::load(base, stride, i, 0, raw);
-        if constexpr (P != 8 && (RECON % 4) != 0) {
-            // trailing 2-real block (recon 18)
-            if constexpr (P == 4) {
+        if constexpr (P == 2) {
+            HLink<RECON> h;
+            h.load(base, stride, i);
+            h.decode(raw);
+        } else {
+            constexpr int NB4 = (P == 8) ? RECON / 2 : RECON / 4;
+            Blocks<P, NB4, true>::load(base, stride, i, 0, raw);
+            if constexpr (P == 4 && (RECON % 4) != 0) {  // trailing 2-real block (recon 18)
                 const float2 *p2 = reinterpret_cast<const float2 *>(reinterpret_cast<const char *>(base) +
                                                                     (size_t)NB4 * 16 * stride);
                 float2 v = ld_stream(p2 + i);
-                raw[RECON - 2] = v.x;
-                raw[RECON - 1] = v.y;
-            } else {
-                const short2 *p2 = reinterpret_cast<const short2 *>(reinterpret_cast<const char *>(base) +
-                                                                    (size_t)NB4 * 8 * stride);
-                const float2 v = dq2(__ldg(reinterpret_cast<const uint32_t *>(p2) + i), kHalfInv);
                 raw[RECON - 2] = v.x;
                 raw[RECON - 1] = v.y;
             }
@@ -410,21 +483,51 @@ struct LinkIO {
 template <int P> struct StoreVec;
 template <> struct StoreVec<8> { using V = double2; };
 template <> struct StoreVec<4> { using V = float4; };
-template <> struct StoreVec<2> { using V = uint2; };
+template <> struct StoreVec<2> { using V = uint4; };
 
-template <int P, int NB>
+// NREAL = 24 (spinor) or 12 (half spinor / face)
+template <int P, int NREAL>
 struct RawVec {
-    using V = typename StoreVec<P>::V;
     using R = typename Prec<P>::R;
-    V d[NB];
-    float n;  // half: the site norm
-    // blocks [b0, b0 + NB) of site i; `norms` = the norm array (half only)
+    static constexpr int RPV = (P == 8) ? 2 : 4;   // reals per stored vector (fp64 / fp32)
+    static constexpr int NB = NREAL / RPV;
+    typename StoreVec<P == 2 ? 4 : P>::V d[P == 2 ? 1 : NB];  // fp64 / fp32 blocks
+    H12 h[NREAL / 12];                                       // half records
+    float n;                                                 // half: the site norm
     template <int MODE>
-    __device__ __forceinline__ void load(const void *base, long stride, long i, int b0, const float *norms) {
+    __device__ __forceinline__ void load_blocks(const void *base, long stride, long i, int b0) {
+        using V = typename StoreVec<P>::V;
         const V *p = reinterpret_cast<const V *>(base);
 #pragma unroll
-        for (int k = 0; k < NB; ++k) d[k] = MODE == 2 ? __ldcg(p + (b0 + k) * stride + i) : __ldg(p + (b0 + k) * stride + i);
-        if constexpr (P == 2) n = MODE == 2 ? __ldcg(norms + i) : __ldg(norms + i);
+        for (int k = 0; k < NB; ++k) d[k] = ld_m<MODE>(p + (b0 + k) * stride + i);
+    }
+    template <int MODE>
+    __device__ __forceinline__ void load_spinor(const void *base, long stride, long i) {
+        if constexpr (P == 2) {
+#pragma unroll
+            for (int hf = 0; hf < 2; ++hf)
+                h[hf].template load<MODE>(cptr(base, h_spinor_u(stride, hf)), cptr(base, h_spinor_v(stride, hf)), i);
+            n = ld_m<MODE>(SpinorIO<2>::norms(base, stride) + i);
+        } else {
+            load_blocks<MODE>(base, stride, i, 0);
+        }
+    }
+    template <int MODE>
+    __device__ __forceinline__ void load_half(const void *base, long stride, long i, int hf) {
+        if constexpr (P == 2) {
+            h[0].template load<MODE>(cptr(base, h_spinor_u(stride, hf)), cptr(base, h_spinor_v(stride, hf)), i);
+            n = ld_m<MODE>(SpinorIO<2>::norms(base, stride) + i);
+        } else {
+            load_blocks<MODE>(base, stride, i, NB * hf);
+        }
+    }
+    __device__ __forceinline__ void load_face(const void *base, long fs, long f) {
+        if constexpr (P == 2) {
+            h[0].template load<0>(base, cptr(base, (size_t)16 * fs), f);
+            n = __ldg(FaceIO<2>::norms(base, fs) + f);
+        } else {
+            load_blocks<0>(base, fs, f, 0);
+        }
     }
     // identical values to SpinorIO / FaceIO loads
     __device__ __forceinline__ void decode(R *out) const {
@@ -442,33 +545,29 @@ struct RawVec {
         } else {
             const float scale = n * kHalfInv;
 #pragma unroll
-            for (int k = 0; k < NB; ++k) {
-                const float2 a = dq2(d[k].x, scale), b = dq2(d[k].y, scale);
-                out[4 * k] = a.x; out[4 * k + 1] = a.y; out[4 * k + 2] = b.x; out[4 * k + 3] = b.y;
-            }
+            for (int r = 0; r < NREAL / 12; ++r) h[r].decode(scale, out + 12 * r);
         }
     }
 };
 
 template <int P, int RECON>
 struct RawLink {
-    using V = typename StoreVec<P>::V;
     using R = typename Prec<P>::R;
     static constexpr int NB = (P == 8) ? RECON / 2 : RECON / 4;
-    static constexpr bool kTail = (P != 8) && (RECON % 4) != 0;
-    V d[NB];
-    typename std::conditional<P == 4, float2, uint32_t>::type tail;
+    static constexpr bool kTail = (P == 4) && (RECON % 4) != 0;
+    typename StoreVec<P == 2 ? 4 : P>::V d[P == 2 ? 1 : NB];
+    float2 tail;
+    HLink<RECON> h;
     __device__ __forceinline__ void load(const void *base, long stride, long i) {
-        const V *p = reinterpret_cast<const V *>(base);
+        if constexpr (P == 2) {
+            h.load(base, stride, i);
+        } else {
+            using V = typename StoreVec<P>::V;
+            const V *p = reinterpret_cast<const V *>(base);
 #pragma unroll
-        for (int k = 0; k < NB; ++k) {
-            if constexpr (P == 2) d[k] = ld_stream_u2(p + k * stride + i);
-            else d[k] = ld_stream(p + k * stride + i);
-        }
-        if constexpr (kTail) {
-            const char *t = reinterpret_cast<const char *>(base) + (size_t)NB * sizeof(V) * stride;
-            if constexpr (P == 4) tail = ld_stream(reinterpret_cast<const float2 *>(t) + i);
-            else tail = __ldg(reinterpret_cast<const uint32_t *>(t) + i);
+            for (int k = 0; k < NB; ++k) d[k] = ld_stream(p + k * stride + i);
+            if constexpr (kTail)
+                tail = ld_stream(reinterpret_cast<const float2 *>(cptr(base, (size_t)NB * sizeof(V) * stride)) + i);
         }
     }
     // identical to LinkIO<P, RECON>::load
@@ -490,16 +589,7 @@ struct RawLink {
                 raw[RECON - 1] = tail.y;
             }
         } else {
-#pragma unroll
-            for (int k = 0; k < NB; ++k) {
-                const float2 a = dq2(d[k].x, kHalfInv), b = dq2(d[k].y, kHalfInv);
-                raw[4 * k] = a.x; raw[4 * k + 1] = a.y; raw[4 * k + 2] = b.x; raw[4 * k + 3] = b.y;
-            }
-            if constexpr (kTail) {
-                const float2 v = dq2(tail, kHalfInv);
-                raw[RECON - 2] = v.x;
-                raw[RECON - 1] = v.y;
-            }
+            h.decode(raw);
         }
         LinkIO<P, RECON>::reconstruct(raw, u);
     }

@@ -198,10 +198,27 @@ struct CloverIO {
         } else if constexpr (P == 4) {
             Blocks<4, 9, true>::load(base, stride, i, 9 * b, m);
         } else {
-            const float2 *nrm = reinterpret_cast<const float2 *>(reinterpret_cast<const char *>(base) +
-                                                                 (size_t)18 * 8 * stride);
-            float2 n = ld_stream(nrm + i);
-            Blocks<2, 9, true>::load(base, stride, i, 9 * b, m, (b ? n.y : n.x) * kHalfInv);
+            // 9 uint4 regions (reals 8k..8k+7); chiral block b = reals 36b..36b+35, so region 4
+            // is split: its low 8 bytes end C+, its high 8 bytes start C-
+            const float2 nn = ld_stream(reinterpret_cast<const float2 *>(cptr(base, (size_t)144 * stride)) + i);
+            const float scale = (b ? nn.y : nn.x) * kHalfInv;
+            uint32_t q[18];
+            const int r0 = b ? 5 : 0;
+#pragma unroll
+            for (int k = 0; k < 4; ++k) {
+                const uint4 w = ld_stream_u4(reinterpret_cast<const uint4 *>(cptr(base, (size_t)16 * (r0 + k) * stride)) + i);
+                const int o = b ? 2 + 4 * k : 4 * k;
+                q[o] = w.x; q[o + 1] = w.y; q[o + 2] = w.z; q[o + 3] = w.w;
+            }
+            const uint2 mid = ld_stream_u2(reinterpret_cast<const uint2 *>(cptr(base, (size_t)64 * stride + 8 * b)) + 2 * i);
+            q[b ? 0 : 16] = mid.x;
+            q[b ? 1 : 17] = mid.y;
+#pragma unroll
+            for (int k = 0; k < 18; ++k) {
+                const float2 d = dq2(q[k], scale);
+                m[2 * k] = d.x;
+                m[2 * k + 1] = d.y;
+            }
         }
     }
 };
@@ -317,16 +334,14 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // of the backward hop are issued before the forward hop is computed: twice the bytes in
     // flight per thread (dslash_pair).
     constexpr bool PAIR = dslash_pair<P, RECON>();
-    constexpr int NBS = (P == 8) ? 12 : 6;  // storage blocks of a spinor
-    const float *nrm = SpinorIO<P>::norms(fin, a.stride);
     auto spatial = [&](auto mu_c, int nf, int nb) {
         constexpr int MU = decltype(mu_c)::value;
-        RawVec<P, NBS> sf, sb;
+        RawVec<P, 24> sf, sb;
         RawLink<P, RECON> lf, lb;
-        sf.template load<INMODE>(fin, a.stride, nf, 0, nrm);
+        sf.template load_spinor<INMODE>(fin, a.stride, nf);
         lf.load(a.gauge[MU][p], a.stride, i);
         if constexpr (PAIR) {
-            sb.template load<INMODE>(fin, a.stride, nb, 0, nrm);
+            sb.template load_spinor<INMODE>(fin, a.stride, nb);
             lb.load(a.gauge[MU][op], a.stride, nb);
         }
         {
@@ -338,7 +353,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             spatial_hop<MU, SF, false>(ps, u, acc);
         }
         if constexpr (!PAIR) {
-            sb.template load<INMODE>(fin, a.stride, nb, 0, nrm);
+            sb.template load_spinor<INMODE>(fin, a.stride, nb);
             lb.load(a.gauge[MU][op], a.stride, nb);
         }
         {
@@ -363,7 +378,6 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         // backward: (1 + SB gamma_4)
         constexpr bool FWD_UPPER = (SF > 0);
         constexpr bool BWD_UPPER = (SB > 0);
-        constexpr int NBH = NBS / 2;
         const int T_loc = a.T_loc;
         // operand addresses first (ghost face / periodic wrap / interior), then one load each
         const bool fwd_ghost = (t == T_loc - 1) && a.ghosted;
@@ -372,19 +386,19 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         const R cb = (t == 0) ? (R)(2.0 * a.bc_back) : (R)2;
         const int nfw = (t == T_loc - 1 ? lex - (T_loc - 1) * XYZ : lex + XYZ) >> 1;
         const int nbw = (t == 0 ? lex + (T_loc - 1) * XYZ : lex - XYZ) >> 1;
-        RawVec<P, NBH> hf, hb;
+        RawVec<P, 12> hf, hb;
         RawLink<P, RECON> lf, lb;
         auto load_f = [&] {
-            if (fwd_ghost) hf.template load<0>(a.ghost_fwd, a.fstride, i - t * a.F, 0, FaceIO<P>::norms(a.ghost_fwd, a.fstride));
-            else hf.template load<INMODE>(fin, a.stride, nfw, FWD_UPPER ? 0 : NBH, nrm);
+            if (fwd_ghost) hf.load_face(a.ghost_fwd, a.fstride, i - t * a.F);
+            else hf.template load_half<INMODE>(fin, a.stride, nfw, FWD_UPPER ? 0 : 1);
             lf.load(a.gauge[3][p], a.stride, i);
         };
         auto load_b = [&] {
             if (bwd_ghost) {
-                hb.template load<0>(a.ghost_back, a.fstride, i, 0, FaceIO<P>::norms(a.ghost_back, a.fstride));
+                hb.load_face(a.ghost_back, a.fstride, i);
                 lb.load(a.gauge_ghost, a.fstride, i);
             } else {
-                hb.template load<INMODE>(fin, a.stride, nbw, BWD_UPPER ? 0 : NBH, nrm);
+                hb.template load_half<INMODE>(fin, a.stride, nbw, BWD_UPPER ? 0 : 1);
                 lb.load(a.gauge[3][op], a.stride, nbw);
             }
         };

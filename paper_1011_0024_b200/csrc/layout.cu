@@ -156,20 +156,18 @@ __device__ void encode_store_link(const double *l /*18*/, void *base, long strid
             q[i] = make_float2((float)raw[RECON - 2], (float)raw[RECON - 1]);
         }
     } else {
-        short4 *p = reinterpret_cast<short4 *>(base);
-        constexpr int NB = RECON / 4;
-        auto q16 = [](double v) { return h16_code(__double2int_rn(v * 32767.0)); };
-        for (int k = 0; k < NB; ++k) {
-            short4 v;
-            v.x = q16(raw[4 * k]); v.y = q16(raw[4 * k + 1]); v.z = q16(raw[4 * k + 2]); v.w = q16(raw[4 * k + 3]);
-            p[k * stride + i] = v;
+        // HLink layout (core.cuh): RECON/8 uint4 regions, then uint2 (RECON%8 == 4), then uint32
+        auto q16 = [](double v) { return (uint32_t)(uint16_t)h16_code(__double2int_rn(v * 32767.0)); };
+        auto w2 = [&](int k) { return q16(raw[k]) | (q16(raw[k + 1]) << 16); };
+        constexpr int N16 = RECON / 8;
+        for (int k = 0; k < N16; ++k)
+            reinterpret_cast<uint4 *>(mptr(base, (size_t)16 * k * stride))[i] = make_uint4(w2(8 * k), w2(8 * k + 2), w2(8 * k + 4), w2(8 * k + 6));
+        size_t off = (size_t)16 * N16 * stride;
+        if constexpr (RECON % 8 >= 4) {
+            reinterpret_cast<uint2 *>(mptr(base, off))[i] = make_uint2(w2(8 * N16), w2(8 * N16 + 2));
+            off += (size_t)8 * stride;
         }
-        if constexpr (RECON % 4) {
-            short2 *q = reinterpret_cast<short2 *>(reinterpret_cast<char *>(base) + (size_t)NB * 8 * stride);
-            short2 v;
-            v.x = q16(raw[RECON - 2]); v.y = q16(raw[RECON - 1]);
-            q[i] = v;
-        }
+        if constexpr (RECON % 4 == 2) reinterpret_cast<uint32_t *>(mptr(base, off))[i] = w2(RECON - 2);
     }
 }
 
@@ -405,23 +403,22 @@ __global__ void k_clover_pack(long Vh, long stride, const double *__restrict__ s
         for (int k = 0; k < 18; ++k)
             p[k * stride + i] = make_float4((float)s[4 * k], (float)s[4 * k + 1], (float)s[4 * k + 2], (float)s[4 * k + 3]);
     } else {
-        short4 *p = reinterpret_cast<short4 *>(dst);
-        float2 *nrm = reinterpret_cast<float2 *>(reinterpret_cast<char *>(dst) + (size_t)18 * 8 * stride);
-        float n[2];
+        // 9 uint4 regions of 8 reals; C+ = reals 0..35 (scale n.x), C- = 36..71 (scale n.y)
+        float2 *nrm = reinterpret_cast<float2 *>(mptr(dst, (size_t)144 * stride));
+        float n[2], inv[2];
         for (int b = 0; b < 2; ++b) {
             double m = 0;
             for (int k = 0; k < 36; ++k) m = fmax(m, fabs(s[36 * b + k]));
             n[b] = (float)m;
-            const float inv = m > 0 ? kHalfMax / (float)m : 0.f;
-            for (int k = 0; k < 9; ++k) {
-                short4 v;
-                v.x = h16_code(__float2int_rn((float)s[36 * b + 4 * k] * inv));
-                v.y = h16_code(__float2int_rn((float)s[36 * b + 4 * k + 1] * inv));
-                v.z = h16_code(__float2int_rn((float)s[36 * b + 4 * k + 2] * inv));
-                v.w = h16_code(__float2int_rn((float)s[36 * b + 4 * k + 3] * inv));
-                p[(9 * b + k) * stride + i] = v;
-            }
+            inv[b] = m > 0 ? kHalfMax / (float)m : 0.f;
         }
+        auto q16 = [&](int k) {
+            return (uint32_t)(uint16_t)h16_code(__float2int_rn((float)s[k] * inv[k >= 36 ? 1 : 0]));
+        };
+        auto w2 = [&](int k) { return q16(k) | (q16(k + 1) << 16); };
+        for (int r = 0; r < 9; ++r)
+            reinterpret_cast<uint4 *>(mptr(dst, (size_t)16 * r * stride))[i] =
+                make_uint4(w2(8 * r), w2(8 * r + 2), w2(8 * r + 4), w2(8 * r + 6));
         nrm[i] = make_float2(n[0], n[1]);
     }
 }
@@ -463,7 +460,7 @@ void launch_clover_apply(int prec, const Geom &g, const void *cl, const void *in
 }
 
 // ============================================================================ faces
-// Raw copy of one 12-real half (3 float4 / 6 double2 / 3 short4 + the site norm): bits only,
+// Raw copy of one 12-real half (3 float4 / 6 double2 / one H12 record + the site norm): bits only,
 // so a partitioned Dslash reads exactly what the unpartitioned one reads.
 template <int P>
 __global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
@@ -484,9 +481,9 @@ __global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int 
         float4 *d = reinterpret_cast<float4 *>(dst);
         for (int b = 0; b < 3; ++b) d[b * fstride + f] = s[(3 * half + b) * stride + i];
     } else {
-        const short4 *s = reinterpret_cast<const short4 *>(in);
-        short4 *d = reinterpret_cast<short4 *>(dst);
-        for (int b = 0; b < 3; ++b) d[b * fstride + f] = s[(3 * half + b) * stride + i];
+        reinterpret_cast<uint4 *>(dst)[f] = reinterpret_cast<const uint4 *>(cptr(in, h_spinor_u(stride, half)))[i];
+        reinterpret_cast<uint2 *>(mptr(dst, (size_t)16 * fstride))[f] =
+            reinterpret_cast<const uint2 *>(cptr(in, h_spinor_v(stride, half)))[i];
         FaceIO<2>::norms(dst, fstride)[f] = SpinorIO<2>::norms(in, stride)[i];
     }
 }
