@@ -59,7 +59,7 @@
 extern "C" {
 #endif
 
-#define QUDAX_ABI_VERSION 1
+#define QUDAX_ABI_VERSION 2
 
 typedef enum {
     QUDAX_OK = 0,
@@ -95,6 +95,22 @@ typedef enum { QUDAX_HOP = 0, QUDAX_CLOVER_INV = 1, QUDAX_CLOVER_XPAY = 2 } quda
  *         one GPU in tests. */
 typedef enum { QUDAX_COMM_NONE = 0, QUDAX_COMM_NCCL = 1, QUDAX_COMM_HOST = 2 } qudax_comm_kind;
 
+/* Spinor halo path of the Dslash when the lattice is split (or in loopback):
+ *   COMM  faces packed into local buffers and moved by the `comm` transport above.
+ *   P2P   kernel-initiated over peer memory (the paper's wish to share
+ *         memory between CUDA and message passing).  The face-pack kernel stores
+ *         the spin-projected faces straight into the T-neighbours' ghost buffers (CUDA IPC
+ *         mappings of their device memory: NVLink/NVSwitch on a multi-GPU node) and then
+ *         raises a sequence flag in the neighbour's memory with a system-scope release; the
+ *         boundary kernel acquires both of its own flags before reading its ghosts.  Nothing is
+ *         enqueued by the host between the kernels and no face is copied twice.  Ghosts are
+ *         double-buffered by sequence parity (a rank can run at most one halo ahead of its
+ *         neighbours, because each boundary kernel waits for both of them).  The IPC handles
+ *         are swapped once at init over `comm` (host_exchange hook or NCCL); gauge-ghost setup
+ *         and global sums keep using `comm`.  With nranks == 1 (comm NONE allowed) the
+ *         neighbour is the rank itself: the loopback test of the kernel path. */
+typedef enum { QUDAX_HALO_COMM = 0, QUDAX_HALO_P2P = 1 } qudax_halo_kind;
+
 typedef struct qudax_ctx qudax_ctx;
 
 /* Host transport hooks for QUDAX_COMM_HOST.  exchange: send send_fwd (bytes) to rank+1 and
@@ -121,6 +137,7 @@ typedef struct {
     qudax_exchange_fn host_exchange; /* QUDAX_COMM_HOST hooks */
     qudax_allreduce_fn host_allreduce;
     void *comm_user;
+    int halo;                    /* qudax_halo_kind (0 = COMM) */
 } qudax_init_param;
 
 typedef struct {

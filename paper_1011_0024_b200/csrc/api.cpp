@@ -238,7 +238,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     DslashArgs args = base_args(c, gc, prec, p, kind, a, reverse);
     args.in = in; args.out = out; args.x = x;
     int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
-    const bool split = (c->comm == QUDAX_COMM_NCCL && c->overlap && g.T_loc > 2);
+    const bool split = (c->comm == QUDAX_COMM_NCCL || c->p2p.on) && c->overlap && g.T_loc > 2;
     const bool multi = (g.nranks > 1);  // cross-rank sums needed before the scalar recurrence
     if (red) {
         QX_CHECK(red->kind != RED_XDOT_NORM || kind == QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
@@ -270,6 +270,34 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         if (!red->S) global_sum(c, c->red_out, 3, red->res);
         else if (multi) device_sum_coef(c, red->S->red, 3, red->S, red->coef_mode);
     };
+    if (c->p2p.on) {  // kernel-initiated halo over peer memory (QUDAX_HALO_P2P)
+        auto &q = c->p2p;
+        const int pi = prec_idx(prec);
+        args.ghosted = 1;
+        args.ghost_back = q.base + q.off_gb[pi];
+        args.ghost_fwd = q.base + q.off_gf[pi];
+        args.p2p_seq = reinterpret_cast<const unsigned *>(q.base + q.off_seq);
+        args.p2p_pdist = (long)q.pdist[pi];
+        unsigned *own_flags = reinterpret_cast<unsigned *>(q.base + q.off_flags);
+        // our t=0 face -> rank-1's ghost_fwd (its flags[1]); t=T_loc-1 face -> rank+1's ghost_back (flags[0])
+        launch_pack_faces_p2p(prec, dagger, g, in, q.peer_back + q.off_gf[pi], q.peer_fwd + q.off_gb[pi], q.pdist[pi],
+                              reinterpret_cast<unsigned *>(q.peer_back + q.off_flags) + 1,
+                              reinterpret_cast<unsigned *>(q.peer_fwd + q.off_flags),
+                              reinterpret_cast<unsigned *>(q.base + q.off_seq),
+                              reinterpret_cast<unsigned *>(q.base + q.off_count), c->stream);
+        c->launches += 1;
+        if (split) {
+            args.p2p_flags = nullptr;  // the interior never touches the ghosts
+            launch(RANGE_INTERIOR, (int)((g.T_loc - 2) * g.F));
+            args.p2p_flags = own_flags;
+            launch(RANGE_BOUNDARY, (int)(2 * g.F));
+        } else {
+            args.p2p_flags = own_flags;
+            launch(RANGE_ALL, (int)g.Vh);
+        }
+        finish_red();
+        return;
+    }
     if (c->comm == QUDAX_COMM_NONE) {
         args.ghosted = 0;
         launch(RANGE_ALL, (int)g.Vh);
@@ -422,7 +450,7 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
         QX_CHECK(out[k] && in[k] && (kind != QUDAX_CLOVER_XPAY || (x && x[k])), QUDAX_ERR_ARG, "null field");
         QX_CHECK(out[k] != in[k], QUDAX_ERR_ARG, "dslash cannot run in place");
     }
-    if (c->comm != QUDAX_COMM_NONE || n == 1) {
+    if (c->comm != QUDAX_COMM_NONE || c->p2p.on || n == 1) {
         for (int k = 0; k < n; ++k)
             dslash_op(c, out[k], in[k], x ? x[k] : nullptr, prec, p, dagger, kind, a, nullptr, reverse);
         return;
@@ -742,6 +770,66 @@ qudax_status qudax_nccl_unique_id(void *out128) {
     return QUDAX_OK;
 }
 
+// QUDAX_HALO_P2P setup: one IPC-exportable region per rank with the same layout everywhere
+// (ctx.h P2P), its handle swapped with both T-neighbours over the comm transport, theirs mapped.
+static void setup_p2p(qudax_ctx *c) {
+    auto &q = c->p2p;
+    const Geom &g = c->g;
+    auto up = [](size_t v) { return (v + 255) & ~(size_t)255; };
+    size_t cur = 0;
+    const int precs[3] = {8, 4, 2};
+    for (int k = 0; k < 3; ++k) {
+        const int pi = prec_idx(precs[k]);
+        q.pdist[pi] = up(face_bytes(precs[k], g.fstride));
+        q.off_gb[pi] = cur;
+        cur += 2 * q.pdist[pi];
+        q.off_gf[pi] = cur;
+        cur += 2 * q.pdist[pi];
+    }
+    q.off_flags = cur;
+    q.off_seq = cur + 64;
+    q.off_count = cur + 128;
+    q.bytes = cur + 256;
+    void *base = nullptr;
+    QX_CUDA(cudaMalloc(&base, q.bytes));  // not the caller's allocator: IPC exports whole allocations
+    q.base = static_cast<char *>(base);
+    QX_CUDA(cudaMemset(q.base, 0, q.bytes));
+    QX_CUDA(cudaDeviceSynchronize());
+    if (g.nranks == 1) {  // loopback: the neighbour is this rank
+        q.peer_back = q.peer_fwd = q.base;
+        return;
+    }
+    static_assert(sizeof(cudaIpcMemHandle_t) == 64, "IPC handle size");
+    cudaIpcMemHandle_t mine, hb, hf;
+    QX_CUDA(cudaIpcGetMemHandle(&mine, q.base));
+    if (c->comm == QUDAX_COMM_HOST) {
+        cudaIpcMemHandle_t s0 = mine, s1 = mine;
+        if (c->host_exchange(&s0, &s1, &hb, &hf, sizeof(mine), c->comm_user))
+            throw Error(QUDAX_ERR_COMM, "host_exchange hook failed (IPC handles)");
+    } else if (c->comm == QUDAX_COMM_NCCL) {
+        char *d = static_cast<char *>(dalloc(c, 3 * sizeof(mine)));
+        QX_CUDA(cudaMemcpyAsync(d, &mine, sizeof(mine), cudaMemcpyHostToDevice, c->stream));
+        exchange(c, d, d, d + 64, d + 128, sizeof(mine), c->stream, nullptr, nullptr, nullptr, nullptr);
+        QX_CUDA(cudaMemcpyAsync(&hb, d + 64, sizeof(mine), cudaMemcpyDeviceToHost, c->stream));
+        QX_CUDA(cudaMemcpyAsync(&hf, d + 128, sizeof(mine), cudaMemcpyDeviceToHost, c->stream));
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+    } else {
+        throw Error(QUDAX_ERR_ARG, "P2P halo with nranks > 1 needs a comm transport for the handle exchange");
+    }
+    void *pb = nullptr;
+    QX_CUDA(cudaIpcOpenMemHandle(&pb, hb, cudaIpcMemLazyEnablePeerAccess));
+    q.peer_back = static_cast<char *>(pb);
+    q.opened_back = true;
+    if (rank_fwd(g) == rank_back(g)) {  // two ranks: one neighbour on both sides
+        q.peer_fwd = q.peer_back;
+    } else {
+        void *pf = nullptr;
+        QX_CUDA(cudaIpcOpenMemHandle(&pf, hf, cudaIpcMemLazyEnablePeerAccess));
+        q.peer_fwd = static_cast<char *>(pf);
+        q.opened_fwd = true;
+    }
+}
+
 qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
     if (!out || !p) return QUDAX_ERR_ARG;
     *out = nullptr;
@@ -751,6 +839,7 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
     if (p->comm == QUDAX_COMM_NCCL && !p->nccl_id) return QUDAX_ERR_ARG;
     if (p->comm == QUDAX_COMM_HOST && (!p->host_exchange || !p->host_allreduce)) return QUDAX_ERR_ARG;
     if (p->comm < 0 || p->comm > 2) return QUDAX_ERR_ARG;
+    if (p->halo != QUDAX_HALO_COMM && p->halo != QUDAX_HALO_P2P) return QUDAX_ERR_ARG;
     auto *c = new qudax_ctx();
     qudax_status st = guard(c, [&] {
         Geom &g = c->g;
@@ -796,6 +885,10 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         const size_t ncount = 2 + (size_t)(g.Vh / 32) / 64 + 64;
         c->d_counter = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * ncount));
         QX_CUDA(cudaMemsetAsync(c->d_counter, 0, sizeof(unsigned) * ncount, c->stream));
+        if (p->halo == QUDAX_HALO_P2P) {
+            setup_p2p(c);
+            c->p2p.on = true;
+        }
     });
     if (st != QUDAX_OK) {
         qudax_finalize(c);
@@ -809,6 +902,9 @@ qudax_status qudax_finalize(qudax_ctx *c) {
     if (!c) return QUDAX_ERR_ARG;
     if (c->stream) cudaStreamSynchronize(c->stream);
     if (c->comm_stream) cudaStreamSynchronize(c->comm_stream);
+    if (c->p2p.opened_fwd) cudaIpcCloseMemHandle(c->p2p.peer_fwd);
+    if (c->p2p.opened_back) cudaIpcCloseMemHandle(c->p2p.peer_back);
+    if (c->p2p.base) cudaFree(c->p2p.base);
     if (c->nccl) ncclCommDestroy(c->nccl);
     for (void *p : c->allocs) {
         if (c->dev_free) c->dev_free(p, c->alloc_user);

@@ -283,7 +283,7 @@ template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) 
 // written by other CTAs earlier in the same launch — the fused Mhat kernel)
 template <int P, int RECON, bool DAG, int KIND, int INMODE = 0>
 __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin, void *fout, const void *fx, int tid,
-                                            double red[3]) {
+                                            double red[3], long goff = 0) {
     using R = typename Prec<P>::R;
     if (a.reverse) tid = a.nthreads - 1 - tid;
     int i;
@@ -389,13 +389,13 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         RawVec<P, 12> hf, hb;
         RawLink<P, RECON> lf, lb;
         auto load_f = [&] {
-            if (fwd_ghost) hf.load_face(a.ghost_fwd, a.fstride, i - t * a.F);
+            if (fwd_ghost) hf.load_face(static_cast<const char *>(a.ghost_fwd) + goff, a.fstride, i - t * a.F);
             else hf.template load_half<INMODE>(fin, a.stride, nfw, FWD_UPPER ? 0 : 1);
             lf.load(a.gauge[3][p], a.stride, i);
         };
         auto load_b = [&] {
             if (bwd_ghost) {
-                hb.load_face(a.ghost_back, a.fstride, i);
+                hb.load_face(static_cast<const char *>(a.ghost_back) + goff, a.fstride, i);
                 lb.load(a.gauge_ghost, a.fstride, i);
             } else {
                 hb.template load_half<INMODE>(fin, a.stride, nbw, BWD_UPPER ? 0 : 1);
@@ -473,6 +473,29 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     }
 }
 
+// Kernel-initiated halo (QUDAX_HALO_P2P): one thread per CTA acquires the two flags the
+// neighbours raise after storing this sequence number's faces into our ghosts (bounded: a
+// broken protocol surfaces as a wrong result, never a hang).  Returns the ghost byte offset of
+// the sequence parity.
+__device__ __forceinline__ unsigned ld_acquire_sys(const unsigned *p) {
+    unsigned v;
+    asm volatile("ld.acquire.sys.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ long p2p_wait(const DslashArgs &a) {
+    __shared__ unsigned s_seq;
+    if (threadIdx.x == 0) {
+        const unsigned s = *reinterpret_cast<const volatile unsigned *>(a.p2p_seq);
+        for (long spin = 0; spin < (1L << 28); ++spin) {
+            if ((int)(ld_acquire_sys(a.p2p_flags) - s) >= 0 && (int)(ld_acquire_sys(a.p2p_flags + 1) - s) >= 0) break;
+            __nanosleep(128);
+        }
+        s_seq = s;
+    }
+    __syncthreads();
+    return (s_seq & 1u) ? a.p2p_pdist : 0L;
+}
+
 template <int P, int RECON, bool DAG, int KIND>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
     // one thread per output site (a one-wave grid-stride variant measured 8-25% slower: the
@@ -489,7 +512,9 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     const void *fin = a.nrhs > 1 ? a.in_m[rhs] : a.in;
     void *fout = a.nrhs > 1 ? a.out_m[rhs] : a.out;
     const void *fx = a.nrhs > 1 ? a.x_m[rhs] : a.x;
-    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND>(a, fin, fout, fx, tid, red);
+    long goff = 0;
+    if (a.p2p_flags) goff = p2p_wait(a);
+    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND>(a, fin, fout, fx, tid, red, goff);
     if (a.red_kind != RED_NONE) reduce_with_tail<3, QX_DSLASH_THREADS>(red, a.tail);
 }
 

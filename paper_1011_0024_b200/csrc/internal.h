@@ -109,6 +109,11 @@ struct DslashArgs {
     const void *clover;    // parity p: T (xpay) or T^{-1} (clover_inv)
     const void *ghost_back; // upper (non-dagger) half-spinors from rank-1, face layout
     const void *ghost_fwd;  // lower (non-dagger) half-spinors from rank+1
+    // kernel-initiated halo: before reading ghosts, wait until p2p_flags[0], p2p_flags[1] >=
+    // *p2p_seq (system-scope acquire); ghosts of odd sequence numbers sit p2p_pdist bytes on
+    const unsigned *p2p_seq;
+    const unsigned *p2p_flags;
+    long p2p_pdist;
     // optional fused reduction over the output (BiCGstab, P:542-558 kernel fusion)
     int red_kind;          // RED_NONE, RED_XDOT_NORM: (<out,x>, |out|^2), RED_RHAT_DOT: <rhat,out>
     RedTail tail;          // 3 sums per CTA; block_offset set per launch (split launches)
@@ -150,6 +155,13 @@ int dslash_blocks_f16(int recon, int dagger, int kind, int nthreads);
 // (upper if !dagger) -> send_fwd.  `in` is the Dslash input field (parity 1-p).
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back,
                        void *send_fwd, cudaStream_t s);
+// kernel-initiated halo (QUDAX_HALO_P2P): the same faces stored straight into the neighbours'
+// ghost buffers dst_back / dst_fwd (+ pdist bytes for odd sequence numbers), then flag_back /
+// flag_fwd (in the neighbours' memory) set to the new sequence number with a system-scope
+// release.  seq / count: this rank's sequence counter and CTA counter (device).
+void launch_pack_faces_p2p(int prec, int dagger, const Geom &g, const void *in, char *dst_back, char *dst_fwd,
+                           size_t pdist, unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count,
+                           cudaStream_t s);
 
 // layout conversion (DR AoS fp64 <-> NR SoA prec), one parity
 void launch_spinor_import(int prec, const Geom &g, int parity, const double *src, void *dst, cudaStream_t s);

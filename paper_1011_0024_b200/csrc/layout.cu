@@ -463,8 +463,9 @@ void launch_clover_apply(int prec, const Geom &g, const void *cl, const void *in
 // Raw copy of one 12-real half (3 float4 / 6 double2 / one H12 record + the site norm): bits only,
 // so a partitioned Dslash reads exactly what the unpartitioned one reads.
 template <int P>
-__global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
-                             const void *__restrict__ in, void *__restrict__ sb, void *__restrict__ sf) {
+__device__ __forceinline__ void k_pack_faces_body(long F, long T_loc, long stride, long fstride, int half_back,
+                                                  int half_fwd, const void *__restrict__ in, void *__restrict__ sb,
+                                                  void *__restrict__ sf) {
     long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
     if (k >= 2 * F) return;
     const bool fwd = k >= F;
@@ -486,6 +487,55 @@ __global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int 
             reinterpret_cast<const uint2 *>(cptr(in, h_spinor_v(stride, half)))[i];
         FaceIO<2>::norms(dst, fstride)[f] = SpinorIO<2>::norms(in, stride)[i];
     }
+}
+template <int P>
+__global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
+                             const void *__restrict__ in, void *__restrict__ sb, void *__restrict__ sf) {
+    k_pack_faces_body<P>(F, T_loc, stride, fstride, half_back, half_fwd, in, sb, sf);
+}
+
+// Kernel-initiated halo: k_pack_faces storing into the neighbours' ghosts (peer memory), then
+// the last CTA raises the neighbours' flags.  Every thread fences its remote stores at system
+// scope before its CTA arrives on the counter, so the flag release orders all of them.
+__device__ __forceinline__ void st_release_sys(unsigned *p, unsigned v) {
+    asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+template <int P>
+__global__ void k_pack_faces_p2p(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
+                                 const void *__restrict__ in, char *dst_back, char *dst_fwd, long pdist,
+                                 unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count) {
+    __shared__ bool last;
+    const unsigned s = *reinterpret_cast<volatile unsigned *>(seq) + 1u;
+    const long off = (s & 1u) ? pdist : 0L;
+    k_pack_faces_body<P>(F, T_loc, stride, fstride, half_back, half_fwd, in, dst_back + off, dst_fwd + off);
+    __threadfence_system();
+    __syncthreads();
+    if (threadIdx.x == 0) last = (atomicAdd(count, 1u) == gridDim.x - 1);
+    __syncthreads();
+    if (last && threadIdx.x == 0) {
+        *count = 0u;
+        *seq = s;
+        __threadfence_system();
+        st_release_sys(flag_back, s);
+        st_release_sys(flag_fwd, s);
+    }
+}
+
+void launch_pack_faces_p2p(int prec, int dagger, const Geom &g, const void *in, char *dst_back, char *dst_fwd,
+                           size_t pdist, unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count,
+                           cudaStream_t s) {
+    const int half_back = dagger ? 0 : 1;
+    const int half_fwd = dagger ? 1 : 0;
+    const int T = 128;
+    const int b = nblk(2 * g.F, T);
+#define QX_PP(P)                                                                                                \
+    k_pack_faces_p2p<P><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, dst_back,   \
+                                        dst_fwd, (long)pdist, flag_back, flag_fwd, seq, count)
+    if (prec == 8) QX_PP(8);
+    else if (prec == 4) QX_PP(4);
+    else QX_PP(2);
+#undef QX_PP
+    QX_CUDA(cudaGetLastError());
 }
 
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back, void *send_fwd,

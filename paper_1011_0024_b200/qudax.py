@@ -21,6 +21,7 @@ HALF, SINGLE, DOUBLE = 2, 4, 8
 EVEN, ODD = 0, 1
 HOP, CLOVER_INV, CLOVER_XPAY = 0, 1, 2
 COMM_NONE, COMM_NCCL, COMM_HOST = 0, 1, 2
+HALO_COMM, HALO_P2P = 0, 1
 PREC_NAMES = {"half": 2, "single": 4, "double": 8, "f16": 2, "f32": 4, "f64": 8}
 
 STATUS = {0: "QUDAX_OK", 1: "QUDAX_ERR_ARG", 2: "QUDAX_ERR_STATE", 3: "QUDAX_ERR_CUDA", 4: "QUDAX_ERR_NCCL",
@@ -46,7 +47,8 @@ class InitParam(ctypes.Structure):
                 ("device", ctypes.c_int), ("comm", ctypes.c_int), ("overlap", ctypes.c_int),
                 ("nccl_id", ctypes.c_void_p), ("stream", ctypes.c_size_t),
                 ("dev_alloc", ALLOC_FN), ("dev_free", FREE_FN), ("alloc_user", ctypes.c_void_p),
-                ("host_exchange", EXCHANGE_FN), ("host_allreduce", ALLREDUCE_FN), ("comm_user", ctypes.c_void_p)]
+                ("host_exchange", EXCHANGE_FN), ("host_allreduce", ALLREDUCE_FN), ("comm_user", ctypes.c_void_p),
+                ("halo", ctypes.c_int)]
 
 
 class GaugeParam(ctypes.Structure):
@@ -234,7 +236,7 @@ class Context:
     spinor_bytes(prec) bytes holding one parity in the library's layout."""
 
     def __init__(self, global_dims, nranks=1, rank=0, device=0, comm=COMM_NONE, overlap=True, nccl_id=None,
-                 stream=None, torch_allocator=True, transport=None):
+                 stream=None, torch_allocator=True, transport=None, halo=HALO_COMM):
         import torch
         self._torch = torch
         self.global_dims = tuple(int(d) for d in global_dims)
@@ -246,6 +248,7 @@ class Context:
         p = InitParam()
         p.global_dims = (ctypes.c_int * 4)(*self.global_dims)
         p.nranks, p.rank, p.device, p.comm, p.overlap = int(nranks), int(rank), self.device, int(comm), int(bool(overlap))
+        p.halo = int(halo)
         self._id = None
         if comm == COMM_NCCL:
             self._id = ctypes.create_string_buffer(bytes(nccl_id), 128)

@@ -31,6 +31,7 @@ def main():
     ap.add_argument("--out", required=True)
     ap.add_argument("--dims", default="8,4,6,16")
     ap.add_argument("--same-gpu", type=int, default=1)
+    ap.add_argument("--halo", default="comm", help="comm | p2p (kernel-initiated over CUDA IPC peer memory)")
     args = ap.parse_args()
     dims = tuple(int(v) for v in args.dims.split(","))
     dist.init_process_group("gloo")
@@ -42,13 +43,15 @@ def main():
     U = qgen.gauge(dims, 1301, eps=-1.0, t_begin=t0, nt=T_loc)
     psi = qgen.spinor(dims, 1302, t_begin=t0, nt=T_loc)
     xin = qgen.spinor(dims, 1303, t_begin=t0, nt=T_loc)
-    result = {"rank": rank, "n": n, "comm": args.comm, "ok": True, "checks": {}}
+    result = {"rank": rank, "n": n, "comm": args.comm, "halo": args.halo, "ok": True, "checks": {}}
+    halo = qudax.HALO_P2P if args.halo == "p2p" else qudax.HALO_COMM
     if args.comm == "nccl":
         obj = [qudax.nccl_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(obj, src=0)
-        ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_NCCL, nccl_id=obj[0])
+        ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_NCCL, nccl_id=obj[0],
+                            halo=halo)
     else:
-        ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_HOST)
+        ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_HOST, halo=halo)
     outs = {}
     for prec, recon in ((8, 18), (4, 12), (2, 12)):
         ctx.gauge_load(U, 0.12, 1.0, prec=prec, recon=recon, t_boundary=-1)

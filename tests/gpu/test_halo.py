@@ -1,6 +1,8 @@
 """Split (halo) path at N=1: faces go pack -> NCCL send/recv to self -> ghost buffers ->
-interior + boundary kernels.  Must be BITWISE equal to the unsplit single-kernel path
-(the exchange moves bits only), overlapped or not, for every precision and dagger."""
+interior + boundary kernels, or (QUDAX_HALO_P2P) the pack kernel stores them straight into the
+ghost buffers and raises the sequence flags the boundary kernel acquires.  Must be BITWISE
+equal to the unsplit single-kernel path (the exchange moves bits only), overlapped or not, for
+every precision and dagger."""
 import numpy as np
 import pytest
 
@@ -12,13 +14,17 @@ pytestmark = pytest.mark.gpu
 
 @pytest.mark.parametrize("prec", [8, 4, 2])
 @pytest.mark.parametrize("overlap", [True, False])
-def test_loopback_bitwise(torch_cuda, prec, overlap):
+@pytest.mark.parametrize("halo", ["nccl", "p2p"])
+def test_loopback_bitwise(torch_cuda, prec, overlap, halo):
     dims = (8, 4, 6, 8)
     U = qgen.gauge(dims, 1201)
     psi = qgen.spinor(dims, 1202)
     x = qgen.spinor(dims, 1203)
     ref = qudax.Context(dims)
-    loop = qudax.Context(dims, comm=qudax.COMM_NCCL, nccl_id=qudax.nccl_unique_id(), overlap=overlap)
+    if halo == "nccl":
+        loop = qudax.Context(dims, comm=qudax.COMM_NCCL, nccl_id=qudax.nccl_unique_id(), overlap=overlap)
+    else:
+        loop = qudax.Context(dims, overlap=overlap, halo=qudax.HALO_P2P)
     for c in (ref, loop):
         c.gauge_load(U, 0.12, 1.0, prec=prec, recon=12)
     outs = {}
@@ -46,3 +52,20 @@ def test_loopback_bitwise(torch_cuda, prec, overlap):
         assert np.array_equal(a, b)
     ref.close()
     loop.close()
+
+
+def test_p2p_loopback_solve(torch_cuda):
+    """Mixed-precision solve through the kernel-initiated halo (graph replay included): same
+    iterations and residual history as the unsplit context (bitwise operators)."""
+    dims = (8, 4, 4, 16)
+    U = qgen.gauge(dims, 1211, eps=0.1)
+    b = qgen.point_source(dims, 0, 0)
+    res = {}
+    for name, kw in (("ref", {}), ("p2p", {"halo": qudax.HALO_P2P})):
+        c = qudax.Context(dims, **kw)
+        c.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+        x, st = c.solve(b, tol=1e-12, delta=0.1, maxiter=1000, prec=8, prec_sloppy=4)
+        res[name] = (x, st)
+        c.close()
+    assert res["ref"][1]["iters"] == res["p2p"][1]["iters"]
+    assert np.array_equal(res["ref"][0], res["p2p"][0])

@@ -24,12 +24,12 @@ def _free_port():
     return p
 
 
-def _run(n, comm, tmp_path, dims):
-    out = tmp_path / f"mp_{comm}_{n}.json"
+def _run(n, comm, tmp_path, dims, halo="comm"):
+    out = tmp_path / f"mp_{comm}_{halo}_{n}.json"
     cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={n}",
            "--master-addr", "127.0.0.1", "--master-port", str(_free_port()),
            os.path.join(HERE, "mp_worker.py"), "--comm", comm, "--out", str(out), "--dims", dims,
-           "--same-gpu", "1" if comm == "host" else "0"]
+           "--same-gpu", "1" if comm == "host" else "0", "--halo", halo]
     r = subprocess.run(cmd, capture_output=True, text=True, timeout=600)
     return r, out
 
@@ -37,6 +37,18 @@ def _run(n, comm, tmp_path, dims):
 @pytest.mark.parametrize("n,dims", [(2, "8,4,6,16"), (4, "8,4,6,16")])
 def test_partitioned_bitwise_host_transport(torch_cuda, tmp_path, n, dims):
     r, out = _run(n, "host", tmp_path, dims)
+    assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
+    res = json.load(open(out))
+    bad = [k for k, v in res["checks"].items() if not v]
+    assert res["ok"], (bad, res.get("solve"))
+
+
+@pytest.mark.parametrize("n", [2, 4])
+def test_partitioned_bitwise_p2p_halo(torch_cuda, tmp_path, n):
+    """Kernel-initiated halo between processes: each rank's pack kernel stores its faces into
+    the neighbours' ghost buffers through CUDA IPC mappings (same GPU here; NVLink peers on a
+    multi-GPU node) and raises their flags; boundary kernels acquire them."""
+    r, out = _run(n, "host", tmp_path, "8,4,6,16", halo="p2p")
     assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
     res = json.load(open(out))
     bad = [k for k, v in res["checks"].items() if not v]

@@ -28,7 +28,7 @@ def test_library_exports_every_header_symbol():
 
 
 def test_abi_version_and_status_strings():
-    assert qudax.lib().qudax_abi_version() == 1
+    assert qudax.lib().qudax_abi_version() == 2
     assert qudax.status_string(0) == "ok"
     assert "unsupported" in qudax.status_string(5)
 
@@ -80,3 +80,31 @@ def test_init_without_gpu_fails_loudly():
     st = qudax.lib().qudax_init(ctypes.byref(h), ctypes.byref(p))
     assert st == 3  # QUDAX_ERR_CUDA: no silent CPU fallback
     assert not h.value
+
+
+def test_binding_struct_layouts_match_header(tmp_path):
+    """The ctypes mirrors of the header's structs have the C compiler's sizes and field offsets
+    (a field added to the header but not to the binding would silently shift every later one)."""
+    import subprocess
+    structs = {"qudax_init_param": qudax.InitParam, "qudax_gauge_param": qudax.GaugeParam,
+               "qudax_solve_param": qudax.SolveParam, "qudax_solve_stats": qudax.SolveStats,
+               "qudax_site_model": qudax.SiteModel, "qudax_kernel_stats": qudax.KernelStats,
+               "qudax_partition": qudax.Partition}
+    lines = ['#include <stdio.h>', '#include <stddef.h>', '#include "qudax.h"', "int main(void) {"]
+    for cname, py in structs.items():
+        lines.append(f'printf("{cname} size %zu\\n", sizeof({cname}));')
+        for f, _ in py._fields_:
+            lines.append(f'printf("{cname} {f} %zu\\n", offsetof({cname}, {f}));')
+    lines += ["return 0;", "}"]
+    src = tmp_path / "layout.c"
+    src.write_text("\n".join(lines))
+    exe = tmp_path / "layout"
+    subprocess.run(["gcc", "-std=c11", "-I", os.path.join(ROOT, "include"), str(src), "-o", str(exe)], check=True)
+    got = {}
+    for ln in subprocess.run([str(exe)], capture_output=True, text=True, check=True).stdout.splitlines():
+        c, f, v = ln.split()
+        got[(c, f)] = int(v)
+    for cname, py in structs.items():
+        assert got[(cname, "size")] == ctypes.sizeof(py), cname
+        for f, _ in py._fields_:
+            assert got[(cname, f)] == getattr(py, f).offset, (cname, f)
