@@ -49,6 +49,8 @@ def parse():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-extra", action="store_true", help="skip the per-precision Dslash table and the config-3 solve")
     ap.add_argument("--overlap", type=int, default=1)
+    ap.add_argument("--halo", default="comm", choices=["comm", "p2p"],
+                    help="N>1 spinor halo: NCCL send/recv (comm) or kernel-initiated over peer memory (p2p)")
     return ap.parse_args()
 
 
@@ -285,7 +287,8 @@ def main():
         obj = [qudax.nccl_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(obj, src=0)
         ctx = qudax.Context(dims, nranks=N, rank=rank, device=local, comm=qudax.COMM_NCCL, nccl_id=obj[0],
-                            overlap=bool(args.overlap))
+                            overlap=bool(args.overlap),
+                            halo=qudax.HALO_P2P if args.halo == "p2p" else qudax.HALO_COMM)
     else:
         ctx = qudax.Context(dims, device=local)
     t0 = rank * T_loc
@@ -416,7 +419,8 @@ def main():
                        "lattice_global": list(dims), "lattice_per_gpu": [SPATIAL, SPATIAL, SPATIAL, T_loc],
                        "precision": {"outer": "f64 recon-18", "sloppy": "f32 recon-12"},
                        "kappa": KAPPA, "csw": CSW, "gauge": f"weak field eps={EPS}", "t_boundary": "antiperiodic",
-                       "delta": 0.1, "parallelism": f"T-slab x{N}" + (" (NCCL halo, overlapped)" if N > 1 else ""),
+                       "delta": 0.1, "parallelism": f"T-slab x{N}" + ((" (P2P kernel-initiated halo)" if args.halo == "p2p" else
+                                                         " (NCCL halo, overlapped)") if N > 1 else ""),
                        "l2": "inputs larger than L2 (>1 GB of gauge+clover+fields per GPU vs 126 MB L2)"},
             "iters_per_step": iters / args.steps, "reliable_updates_per_step": updates / args.steps,
             "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches, "clocks": clocks,

@@ -238,7 +238,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     DslashArgs args = base_args(c, gc, prec, p, kind, a, reverse);
     args.in = in; args.out = out; args.x = x;
     int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
-    const bool split = (c->comm == QUDAX_COMM_NCCL || c->p2p.on) && c->overlap && g.T_loc > 2;
+    const bool split = c->comm == QUDAX_COMM_NCCL && !c->p2p.on && c->overlap && g.T_loc > 2;
     const bool multi = (g.nranks > 1);  // cross-rank sums needed before the scalar recurrence
     if (red) {
         QX_CHECK(red->kind != RED_XDOT_NORM || kind == QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
@@ -276,22 +276,33 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         args.ghosted = 1;
         args.ghost_back = q.base + q.off_gb[pi];
         args.ghost_fwd = q.base + q.off_gf[pi];
-        args.p2p_seq = reinterpret_cast<const unsigned *>(q.base + q.off_seq);
+        args.p2p_cseq = reinterpret_cast<unsigned *>(q.base + q.off_cseq);
+        args.p2p_ccount = reinterpret_cast<unsigned *>(q.base + q.off_ccount);
         args.p2p_pdist = (long)q.pdist[pi];
         unsigned *own_flags = reinterpret_cast<unsigned *>(q.base + q.off_flags);
         // our t=0 face -> rank-1's ghost_fwd (its flags[1]); t=T_loc-1 face -> rank+1's ghost_back (flags[0])
-        launch_pack_faces_p2p(prec, dagger, g, in, q.peer_back + q.off_gf[pi], q.peer_fwd + q.off_gb[pi], q.pdist[pi],
-                              reinterpret_cast<unsigned *>(q.peer_back + q.off_flags) + 1,
-                              reinterpret_cast<unsigned *>(q.peer_fwd + q.off_flags),
-                              reinterpret_cast<unsigned *>(q.base + q.off_seq),
-                              reinterpret_cast<unsigned *>(q.base + q.off_count), c->stream);
-        c->launches += 1;
-        if (split) {
-            args.p2p_flags = nullptr;  // the interior never touches the ghosts
-            launch(RANGE_INTERIOR, (int)((g.T_loc - 2) * g.F));
+        auto pack = [&](cudaStream_t st) {
+            launch_pack_faces_p2p(prec, dagger, g, in, q.peer_back + q.off_gf[pi], q.peer_fwd + q.off_gb[pi],
+                                  q.pdist[pi], reinterpret_cast<unsigned *>(q.peer_back + q.off_flags) + 1,
+                                  reinterpret_cast<unsigned *>(q.peer_fwd + q.off_flags),
+                                  reinterpret_cast<unsigned *>(q.base + q.off_seq),
+                                  reinterpret_cast<unsigned *>(q.base + q.off_count), st);
+            c->launches += 1;
+        };
+        if (c->overlap && g.T_loc > 2) {
+            // ONE Dslash launch (RANGE_TAIL) beside the pack on the high-priority comm stream:
+            // interior CTAs first, the boundary CTAs at the grid's tail acquire the neighbours'
+            // flags.  The join after it only keeps `in` alive until our own pack has read it.
+            QX_CUDA(cudaEventRecord(c->ev_in, c->stream));
+            QX_CUDA(cudaStreamWaitEvent(c->comm_stream, c->ev_in, 0));
+            pack(c->comm_stream);
+            QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
             args.p2p_flags = own_flags;
-            launch(RANGE_BOUNDARY, (int)(2 * g.F));
+            args.reverse = 0;  // the waiting CTAs must be the last ones
+            launch(RANGE_TAIL, (int)g.Vh);
+            QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
         } else {
+            pack(c->stream);
             args.p2p_flags = own_flags;
             launch(RANGE_ALL, (int)g.Vh);
         }
@@ -789,7 +800,9 @@ static void setup_p2p(qudax_ctx *c) {
     q.off_flags = cur;
     q.off_seq = cur + 64;
     q.off_count = cur + 128;
-    q.bytes = cur + 256;
+    q.off_cseq = cur + 192;
+    q.off_ccount = cur + 256;
+    q.bytes = cur + 512;
     void *base = nullptr;
     QX_CUDA(cudaMalloc(&base, q.bytes));  // not the caller's allocator: IPC exports whole allocations
     q.base = static_cast<char *>(base);

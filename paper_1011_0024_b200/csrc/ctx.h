@@ -84,14 +84,15 @@ struct qudax_ctx {
     // kernel-initiated halo over peer memory (QUDAX_HALO_P2P).  One cudaMalloc region per rank,
     // identical layout on every rank: per precision ghost_back[2], ghost_fwd[2] (sequence
     // parity), then flags[2] (flags[0] raised by rank-1 after it filled ghost_back, flags[1] by
-    // rank+1 after ghost_fwd), the local sequence counter and the pack kernel's CTA counter.
+    // rank+1 after ghost_fwd), the producer (pack) and consumer (Dslash) halo counters and
+    // their CTA counters.
     struct P2P {
         bool on = false;
         char *base = nullptr;                       // own region (cudaMalloc, IPC-exported)
         char *peer_back = nullptr, *peer_fwd = nullptr;  // neighbours' regions (IPC-mapped or own)
         bool opened_back = false, opened_fwd = false;
         size_t off_gb[3] = {}, off_gf[3] = {}, pdist[3] = {};
-        size_t off_flags = 0, off_seq = 0, off_count = 0, bytes = 0;
+        size_t off_flags = 0, off_seq = 0, off_count = 0, off_cseq = 0, off_ccount = 0, bytes = 0;
     } p2p;
 
     // workspace

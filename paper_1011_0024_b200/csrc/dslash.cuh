@@ -289,6 +289,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     int i;
     if (a.range == RANGE_ALL) i = tid;
     else if (a.range == RANGE_INTERIOR) i = a.F + tid;
+    else if (a.range == RANGE_TAIL) {
+        const int ni = (a.T_loc - 2) * a.F;
+        const int j = tid - ni;
+        i = (tid < ni) ? a.F + tid : ((j < a.F) ? j : (a.T_loc - 1) * a.F + (j - a.F));
+    }
     else i = (tid < a.F) ? tid : (a.T_loc - 1) * a.F + (tid - a.F);
 
     const int X = a.X, Y = a.Y, Z = a.Z, Xh = a.Xh;
@@ -485,7 +490,7 @@ __device__ __forceinline__ unsigned ld_acquire_sys(const unsigned *p) {
 __device__ __forceinline__ long p2p_wait(const DslashArgs &a) {
     __shared__ unsigned s_seq;
     if (threadIdx.x == 0) {
-        const unsigned s = *reinterpret_cast<const volatile unsigned *>(a.p2p_seq);
+        const unsigned s = *reinterpret_cast<const volatile unsigned *>(a.p2p_cseq) + 1u;
         for (long spin = 0; spin < (1L << 28); ++spin) {
             if ((int)(ld_acquire_sys(a.p2p_flags) - s) >= 0 && (int)(ld_acquire_sys(a.p2p_flags + 1) - s) >= 0) break;
             __nanosleep(128);
@@ -513,8 +518,16 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     void *fout = a.nrhs > 1 ? a.out_m[rhs] : a.out;
     const void *fx = a.nrhs > 1 ? a.x_m[rhs] : a.x;
     long goff = 0;
-    if (a.p2p_flags) goff = p2p_wait(a);
+    // RANGE_TAIL: only CTAs holding boundary sites (the grid's last ones) wait for the halo
+    if (a.p2p_flags && (a.range != RANGE_TAIL || (blk + 1) * (int)blockDim.x > (a.T_loc - 2) * a.F)) goff = p2p_wait(a);
     if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND>(a, fin, fout, fx, tid, red, goff);
+    if (a.p2p_flags) {  // the last CTA to finish advances the consumed-halo counter
+        __syncthreads();
+        if (threadIdx.x == 0 && atomicAdd(a.p2p_ccount, 1u) == gridDim.x - 1) {
+            *a.p2p_ccount = 0u;
+            *a.p2p_cseq += 1u;
+        }
+    }
     if (a.red_kind != RED_NONE) reduce_with_tail<3, QX_DSLASH_THREADS>(red, a.tail);
 }
 

@@ -87,7 +87,10 @@ struct RedTail {
 };
 
 // ----------------------------------------------------------------------------- kernels
-enum SiteRange { RANGE_ALL = 0, RANGE_INTERIOR = 1, RANGE_BOUNDARY = 2 };
+// RANGE_TAIL: every site, interior first and the 2F boundary sites in the LAST CTAs of the
+// grid, which alone wait for the kernel-initiated halo (one launch: the interior overlaps the
+// peers' face stores, the boundary fills the grid's tail)
+enum SiteRange { RANGE_ALL = 0, RANGE_INTERIOR = 1, RANGE_BOUNDARY = 2, RANGE_TAIL = 3 };
 constexpr int kMaxRhs = 8;
 
 struct DslashArgs {
@@ -109,9 +112,13 @@ struct DslashArgs {
     const void *clover;    // parity p: T (xpay) or T^{-1} (clover_inv)
     const void *ghost_back; // upper (non-dagger) half-spinors from rank-1, face layout
     const void *ghost_fwd;  // lower (non-dagger) half-spinors from rank+1
-    // kernel-initiated halo: before reading ghosts, wait until p2p_flags[0], p2p_flags[1] >=
-    // *p2p_seq (system-scope acquire); ghosts of odd sequence numbers sit p2p_pdist bytes on
-    const unsigned *p2p_seq;
+    // kernel-initiated halo: this launch consumes halo number s = *p2p_cseq + 1: before reading
+    // ghosts its boundary CTAs wait until p2p_flags[0], p2p_flags[1] >= s (system-scope
+    // acquire); ghosts of odd s sit p2p_pdist bytes on.  The launch's last CTA (counter
+    // p2p_ccount) advances *p2p_cseq.  The pack kernel keeps its own producer counter, so the
+    // two may run concurrently.
+    unsigned *p2p_cseq;
+    unsigned *p2p_ccount;
     const unsigned *p2p_flags;
     long p2p_pdist;
     // optional fused reduction over the output (BiCGstab, P:542-558 kernel fusion)

@@ -495,8 +495,9 @@ __global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int 
 }
 
 // Kernel-initiated halo: k_pack_faces storing into the neighbours' ghosts (peer memory), then
-// the last CTA raises the neighbours' flags.  Every thread fences its remote stores at system
-// scope before its CTA arrives on the counter, so the flag release orders all of them.
+// the last CTA raises the neighbours' flags.  Each CTA's stores are ordered before its arrival
+// on the counter by bar.sync + one system-scope fence (cumulative, as in a grid barrier), and
+// the last CTA's fence + release orders all of them before the flags.
 __device__ __forceinline__ void st_release_sys(unsigned *p, unsigned v) {
     asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
@@ -508,9 +509,11 @@ __global__ void k_pack_faces_p2p(long F, long T_loc, long stride, long fstride, 
     const unsigned s = *reinterpret_cast<volatile unsigned *>(seq) + 1u;
     const long off = (s & 1u) ? pdist : 0L;
     k_pack_faces_body<P>(F, T_loc, stride, fstride, half_back, half_fwd, in, dst_back + off, dst_fwd + off);
-    __threadfence_system();
     __syncthreads();
-    if (threadIdx.x == 0) last = (atomicAdd(count, 1u) == gridDim.x - 1);
+    if (threadIdx.x == 0) {
+        __threadfence_system();
+        last = (atomicAdd(count, 1u) == gridDim.x - 1);
+    }
     __syncthreads();
     if (last && threadIdx.x == 0) {
         *count = 0u;
