@@ -191,6 +191,22 @@ class WilsonClover:
     def mdagm(self, x_e):
         return self.matpc(self.matpc(x_e), dagger=True)
 
+    def matpc_sym(self, x_e, dagger=False):
+        """Symmetric Schur complement (the other form of P:190-195):
+        Mhat_sym x_e = x_e - kappa^2 T_ee^{-1} D_eo T_oo^{-1} D_oe x_e (even sites), i.e.
+        T_ee^{-1} (M_ee - M_eo M_oo^{-1} M_oe).  dagger: the explicit adjoint
+        x_e - kappa^2 (D^dag)_eo T_oo^{-1} (D^dag)_oe T_ee^{-1} x_e (T Hermitian)."""
+        if not dagger:
+            tmp = self.Tinv_pp(self.Dpq(x_e, 1), 1)
+            return restrict(x_e, 0) - self.kappa ** 2 * self.Tinv_pp(self.Dpq(tmp, 0), 0)
+        y = self.Tinv_pp(x_e, 0)
+        tmp = self.Tinv_pp(self.Dpq(y, 1, True), 1)
+        return restrict(x_e, 0) - self.kappa ** 2 * self.Dpq(tmp, 0, True)
+
+    def prepare_sym(self, b):
+        """Source of the symmetric system: T_ee^{-1} (b_e + kappa D_eo T_oo^{-1} b_o)."""
+        return self.Tinv_pp(self.prepare(b), 0)
+
     def prepare(self, b):
         b_e, b_o = restrict(b, 0), restrict(b, 1)
         return b_e + self.kappa * self.Dpq(self.Tinv_pp(b_o, 1), 0)
