@@ -82,8 +82,10 @@ typedef enum { QUDAX_EVEN = 0, QUDAX_ODD = 1 } qudax_parity;
  *   CLOVER_INV  out = T_pp^{-1} D_{p,1-p} in                         (+504, clover fused,
  *                                                                      P:390-395)
  *   CLOVER_XPAY out = T_pp x + a * D_{p,1-p} in                     (+504 +48)
- * Mhat = [kernel CLOVER_INV on odd] then [kernel CLOVER_XPAY on even, a = -kappa^2]. */
-typedef enum { QUDAX_HOP = 0, QUDAX_CLOVER_INV = 1, QUDAX_CLOVER_XPAY = 2 } qudax_dslash_kind;
+ *   CLOVER_INV_XPAY out = x + a * T_pp^{-1} D_{p,1-p} in            (+504 +48)
+ * Mhat = [kernel CLOVER_INV on odd] then [kernel CLOVER_XPAY on even, a = -kappa^2];
+ * the symmetric form T_ee^{-1} Mhat ends with CLOVER_INV_XPAY instead. */
+typedef enum { QUDAX_HOP = 0, QUDAX_CLOVER_INV = 1, QUDAX_CLOVER_XPAY = 2, QUDAX_CLOVER_INV_XPAY = 3 } qudax_dslash_kind;
 
 /* Halo transport:
  *   NONE  nranks must be 1; the Dslash wraps T periodically inside one kernel.
@@ -153,7 +155,9 @@ typedef struct {
     int maxiter;                 /* iteration cap; tol = 0 with maxiter = k runs exactly k iterations */
     int prec_sloppy;             /* precision of the Krylov iteration (must have a gauge copy) */
     int prec;                    /* outer precision of x, r and the reliable-update residual */
-    int use_schur;               /* 1: solve the full system M x = b via prepare/Mhat/reconstruct */
+    int use_schur;               /* 1: solve the full system M x = b via prepare/Mhat/reconstruct with the
+                                    asymmetric Schur form; 2: the same with the symmetric form
+                                    (qudax_matpc_sym); 0: solve Mhat x_e = b_e only */
     double *res_history;         /* optional host array: ||r_k|| / ||bhat|| after iteration k (the
                                     iterated residual, replaced by the true one at reliable updates) */
     int history_cap;             /* capacity of res_history (0 = none) */
@@ -250,6 +254,11 @@ qudax_status qudax_dslash(qudax_ctx *ctx, void *out, const void *in, const void 
                           int out_parity, int dagger, int kind, double a);
 /* out_e = Mhat in_e (dagger = 0) or Mhat^dag in_e (dagger = 1); 2 Dslash kernels + 2 halos. */
 qudax_status qudax_matpc(qudax_ctx *ctx, void *out, const void *in, int prec, int dagger);
+/* Symmetric Schur form: out_e = in_e - kappa^2 T_ee^{-1} D_eo T_oo^{-1} D_oe in_e
+ * = T_ee^{-1} Mhat in_e — kernels CLOVER_INV then CLOVER_INV_XPAY; dagger = 1 applies the explicit
+ * adjoint in_e - kappa^2 (D^dag)_eo T_oo^{-1} (D^dag)_oe T_ee^{-1} in_e (clover apply, CLOVER_INV,
+ * HOP and an xpay: it is not gamma5-Hermitian, so no dagger-by-flag shortcut). */
+qudax_status qudax_matpc_sym(qudax_ctx *ctx, void *out, const void *in, int prec, int dagger);
 /* Multi-RHS forms (the paper's production calls the solver for many
  * right-hand sides per configuration): nrhs (1..8) independent fields
  * in one launch that streams the links and clover from HBM about once for all of them.

@@ -169,7 +169,7 @@ static void rec_model(const qudax_ctx::TimingRec &r, qudax_site_model *out) {
     qudax_model(r.prec, r.recon, r.kind, &m);
     const double w = r.prec, nrm = (r.prec == 2) ? 4 : 0;
     const double sp = 24 * w + nrm;
-    const double per_rhs = (r.kind == QUDAX_CLOVER_XPAY ? 3 : 2) * sp;  // in, out (, x)
+    const double per_rhs = (r.kind >= QUDAX_CLOVER_XPAY ? 3 : 2) * sp;  // in, out (, x)
     (void)hop;
     out->flops = m.flops * r.sites * r.nrhs;
     out->bytes_compulsory = ((m.bytes_compulsory - per_rhs) + per_rhs * r.nrhs) * r.sites;
@@ -230,8 +230,8 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
                double a, const RedReq *red, int reverse) {
     check_prec(prec);
     QX_CHECK(p == 0 || p == 1, QUDAX_ERR_ARG, "parity must be 0 or 1");
-    QX_CHECK(kind >= 0 && kind <= 2, QUDAX_ERR_ARG, "bad dslash kind");
-    QX_CHECK(out && in && (kind != QUDAX_CLOVER_XPAY || x), QUDAX_ERR_ARG, "null field");
+    QX_CHECK(kind >= 0 && kind <= 3, QUDAX_ERR_ARG, "bad dslash kind");
+    QX_CHECK(out && in && (kind < QUDAX_CLOVER_XPAY || x), QUDAX_ERR_ARG, "null field");
     QX_CHECK(out != in, QUDAX_ERR_ARG, "dslash cannot run in place");
     auto &gc = gauge_for(c, prec);
     const Geom &g = c->g;
@@ -241,7 +241,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     const bool split = c->comm == QUDAX_COMM_NCCL && !c->p2p.on && c->overlap && g.T_loc > 2;
     const bool multi = (g.nranks > 1);  // cross-rank sums needed before the scalar recurrence
     if (red) {
-        QX_CHECK(red->kind != RED_XDOT_NORM || kind == QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
+        QX_CHECK(red->kind != RED_XDOT_NORM || kind >= QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
         QX_CHECK(red->kind != RED_RHAT_DOT || red->rhat, QUDAX_ERR_ARG, "rhat-dot needs rhat");
         // CTA slots of up to two launches + their group slots (reduce.cuh)
         if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / 32) + 64)));
@@ -435,7 +435,34 @@ static void matpc_fused(qudax_ctx *c, void *out, const void *in, void *t, int pr
     if (red && !red->S) global_sum(c, c->red_out, 3, red->res);
 }
 
+// symmetric Schur form: T_ee^{-1} Mhat.  Non-dagger: CLOVER_INV on odd,
+// CLOVER_INV_XPAY on even (fused reductions as for Mhat).  Dagger (explicit adjoint, not
+// gamma5-Hermitian): T_ee^{-1} in -> CLOVER_INV^dag on odd -> HOP^dag on even -> in - kappa^2 (.)
+void matpc_sym_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red) {
+    void *t = tmp_odd(c, prec);
+    if (!dagger) {
+        dslash_op(c, t, in, nullptr, prec, 1, 0, QUDAX_CLOVER_INV, 0.0, nullptr);
+        dslash_op(c, out, t, in, prec, 0, 0, QUDAX_CLOVER_INV_XPAY, -c->kappa * c->kappa, red, 1);
+        return;
+    }
+    QX_CHECK(!red, QUDAX_ERR_ARG, "symmetric Mhat^dag: no fused reductions");
+    QX_CHECK(out != in, QUDAX_ERR_ARG, "matpc_sym dagger cannot run in place");
+    auto &ys = c->tmp_sym[prec_idx(prec)];
+    if (!ys) ys = dalloc(c, spinor_bytes(prec, c->g.stride));
+    void *y = ys;
+    clover_apply_op(c, y, in, prec, 0, true);
+    dslash_op(c, t, y, nullptr, prec, 1, 1, QUDAX_CLOVER_INV, 0.0, nullptr);
+    dslash_op(c, y, t, nullptr, prec, 0, 1, QUDAX_HOP, 0.0, nullptr);
+    void *f[3] = {const_cast<void *>(in), y, out};
+    const double a = -c->kappa * c->kappa;
+    blas_op(c, OP_XPAY, prec, f, &a, nullptr);
+}
+
 void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red) {
+    if (c->matpc_sym) {
+        matpc_sym_op(c, out, in, prec, dagger, red);
+        return;
+    }
     void *t = tmp_odd(c, prec);
     if (c->comm == QUDAX_COMM_NONE && c->fused && c->g.T_loc >= 2) {
         matpc_fused(c, out, in, t, prec, dagger, red);
@@ -456,9 +483,9 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
     check_prec(prec);
     QX_CHECK(n >= 1 && n <= kMaxRhs, QUDAX_ERR_ARG, "nrhs must be 1.." + std::to_string(kMaxRhs));
     QX_CHECK(p == 0 || p == 1, QUDAX_ERR_ARG, "parity must be 0 or 1");
-    QX_CHECK(kind >= 0 && kind <= 2, QUDAX_ERR_ARG, "bad dslash kind");
+    QX_CHECK(kind >= 0 && kind <= 3, QUDAX_ERR_ARG, "bad dslash kind");
     for (int k = 0; k < n; ++k) {
-        QX_CHECK(out[k] && in[k] && (kind != QUDAX_CLOVER_XPAY || (x && x[k])), QUDAX_ERR_ARG, "null field");
+        QX_CHECK(out[k] && in[k] && (kind < QUDAX_CLOVER_XPAY || (x && x[k])), QUDAX_ERR_ARG, "null field");
         QX_CHECK(out[k] != in[k], QUDAX_ERR_ARG, "dslash cannot run in place");
     }
     if (c->comm != QUDAX_COMM_NONE || c->p2p.on || n == 1) {
@@ -742,15 +769,15 @@ qudax_status qudax_partition_info(const int global_dims[4], int nranks, int rank
 
 qudax_status qudax_model(int prec, int recon, int kind, qudax_site_model *o) {
     if (!o || (prec != 2 && prec != 4 && prec != 8) || (recon != 18 && recon != 12 && recon != 8) || kind < -2 ||
-        kind > 2)
+        kind > 3)
         return QUDAX_ERR_ARG;
     const double w = prec;
     const double norm = (prec == 2) ? 4 : 0;
     const double sp = 24 * w + norm, hsp = 12 * w + norm, link = recon * w, clov = 72 * w + (prec == 2 ? 8 : 0);
     auto one = [&](int k, qudax_site_model *m) {
         const double cl = (k == QUDAX_HOP) ? 0 : clov;
-        const double xs = (k == QUDAX_CLOVER_XPAY) ? sp : 0;
-        m->flops = 1320 + (k == QUDAX_HOP ? 0 : 504) + (k == QUDAX_CLOVER_XPAY ? 48 : 0);
+        const double xs = (k >= QUDAX_CLOVER_XPAY) ? sp : 0;
+        m->flops = 1320 + (k == QUDAX_HOP ? 0 : 504) + (k >= QUDAX_CLOVER_XPAY ? 48 : 0);
         m->bytes_paper = 6 * sp + 2 * hsp + 8 * link + cl + xs + sp;
         m->bytes_compulsory = 8 * link + sp + cl + xs + sp;
     };
@@ -1101,6 +1128,15 @@ qudax_status qudax_matpc(qudax_ctx *c, void *out, const void *in, int prec, int 
     return guard(c, [&] {
         QX_CHECK(out && in && out != in, QUDAX_ERR_ARG, "matpc: bad fields");
         matpc_op(c, out, in, prec, dagger ? 1 : 0);
+    });
+}
+
+qudax_status qudax_matpc_sym(qudax_ctx *c, void *out, const void *in, int prec, int dagger) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        QX_CHECK(out && in && out != in, QUDAX_ERR_ARG, "matpc_sym: bad fields");
+        check_prec(prec);
+        matpc_sym_op(c, out, in, prec, dagger ? 1 : 0, nullptr);
     });
 }
 

@@ -52,6 +52,9 @@ struct qudax_ctx {
     // measured slower than the two kernels (L2 kept only ~1/3 of the reusable bytes, plus
     // dependency waits) — profiles/r01_fused_matpc.md
     bool fused = false;
+    // the Schur form matpc_op applies: 0 asymmetric (default), 1 symmetric (set by a solve with
+    // use_schur = 2 for its duration, and by qudax_matpc_sym)
+    int matpc_sym = 0;
     const int *fstages = nullptr;
     unsigned *fcounters = nullptr;
     qx::SolverScalars *d_scal = nullptr, *h_scal = nullptr;
@@ -96,7 +99,7 @@ struct qudax_ctx {
     } p2p;
 
     // workspace
-    void *tmp_odd[3] = {}, *tmp_even[3] = {};
+    void *tmp_odd[3] = {}, *tmp_even[3] = {}, *tmp_sym[3] = {};
     void *tmp_multi[3][qx::kMaxRhs] = {};
     double *partials = nullptr, *red_out = nullptr, *h_red = nullptr;
     double *dpart = nullptr;  // per-CTA partials of Dslash-fused reductions
@@ -129,6 +132,7 @@ struct RedReq {
 void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
                double a, const RedReq *red = nullptr, int reverse = 0);
 void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr);
+void matpc_sym_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr);
 void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, const void *const *x, int n, int prec,
                      int p, int dagger, int kind, double a, int reverse);
 void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger);

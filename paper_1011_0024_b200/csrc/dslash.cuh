@@ -435,6 +435,17 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             for (int c = 0; c < 3; ++c) res[s][c] = acc[s][c];
     } else if constexpr (KIND == QUDAX_CLOVER_INV) {
         apply_clover<P>(a.clover, a.stride, i, acc, res);
+    } else if constexpr (KIND == QUDAX_CLOVER_INV_XPAY) {  // symmetric Schur: out = x + a T^{-1} D in
+        Cx<R> ti[4][3], xs[4][3];
+        apply_clover<P>(a.clover, a.stride, i, acc, ti);
+        R v[24];
+        SpinorIO<P>::load(fx, a.stride, i, v);
+        unpack_spinor(v, xs);
+        const R co = (R)a.a;
+#pragma unroll
+        for (int s = 0; s < 4; ++s)
+#pragma unroll
+            for (int c = 0; c < 3; ++c) res[s][c] = axpy(co, ti[s][c], xs[s][c]);
     } else if (xpay_early) {
         const R co = (R)a.a;
 #pragma unroll
@@ -540,7 +551,7 @@ template <int P>
 int dslash_blocks_prec(int recon, int dagger, int kind, int nthreads) {
 #define QX_DB(RC, DG, KD) \
     if (recon == RC && dagger == DG && kind == KD) return dslash_blocks<P, RC, DG, KD>(nthreads);
-#define QX_DB_K(RC, DG) QX_DB(RC, DG, 0) QX_DB(RC, DG, 1) QX_DB(RC, DG, 2)
+#define QX_DB_K(RC, DG) QX_DB(RC, DG, 0) QX_DB(RC, DG, 1) QX_DB(RC, DG, 2) QX_DB(RC, DG, 3)
 #define QX_DB_D(RC) QX_DB_K(RC, false) QX_DB_K(RC, true)
     QX_DB_D(18) QX_DB_D(12) QX_DB_D(8)
 #undef QX_DB_D
@@ -559,7 +570,7 @@ void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cu
                                        threads, 0, s>>>(a);                                     \
         return;                                                                                 \
     }
-#define QX_DS_K(RC, DG) QX_DS(RC, DG, 0) QX_DS(RC, DG, 1) QX_DS(RC, DG, 2)
+#define QX_DS_K(RC, DG) QX_DS(RC, DG, 0) QX_DS(RC, DG, 1) QX_DS(RC, DG, 2) QX_DS(RC, DG, 3)
 #define QX_DS_D(RC) QX_DS_K(RC, false) QX_DS_K(RC, true)
     QX_DS_D(18) QX_DS_D(12) QX_DS_D(8)
 #undef QX_DS_D

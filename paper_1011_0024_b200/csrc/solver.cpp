@@ -89,8 +89,17 @@ static cudaGraphExec_t capture_graph(qudax_ctx *c, F &&body, long long *nlaunch)
     return exec;
 }
 
+// the Schur form matpc_op applies during one solve (restored on every exit path)
+struct SchurForm {
+    qudax_ctx *c;
+    int saved;
+    SchurForm(qudax_ctx *c_, bool sym) : c(c_), saved(c_->matpc_sym) { c->matpc_sym = sym ? 1 : 0; }
+    ~SchurForm() { c->matpc_sym = saved; }
+};
+
 // b (device fp64 DR slab) -> b_e, b_o and the Schur source
-//   bhat = b_e + kappa D_eo T_oo^{-1} b_o   (use_schur), else bhat = b_e
+//   bhat = b_e + kappa D_eo T_oo^{-1} b_o   (use_schur = 1), T_ee^{-1} of that (use_schur = 2,
+//   symmetric form), else bhat = b_e
 static void prepare_source(qudax_ctx *c, int Pd, const double *b_dev, void *b_e, void *b_o, void *bh, void *t_e,
                            void *t_o, int use_schur) {
     const Geom &g = c->g;
@@ -103,6 +112,10 @@ static void prepare_source(qudax_ctx *c, int Pd, const double *b_dev, void *b_e,
         void *f[3] = {b_e, t_e, bh};
         double a = c->kappa;
         blas_op(c, OP_XPAY, Pd, f, &a, nullptr);                   // bhat = b_e + kappa (...)
+        if (use_schur == 2) {                                          // symmetric: T_ee^{-1} bhat
+            clover_apply_op(c, t_e, bh, Pd, 0, true);
+            copy(c, bh, t_e, Pd);
+        }
     } else {
         copy(c, bh, b_e, Pd);
     }
@@ -149,6 +162,8 @@ static void finish_solution(qudax_ctx *c, int Pd, double *x_dev, void *b_e, void
 }
 
 void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *sp, qudax_solve_stats *st) {
+    QX_CHECK(sp->use_schur >= 0 && sp->use_schur <= 2, QUDAX_ERR_ARG, "use_schur must be 0, 1 or 2");
+    SchurForm form_guard(c, sp->use_schur == 2);
     QX_CHECK(c->gauge_loaded, QUDAX_ERR_STATE, "gauge not loaded");
     const int Pd = sp->prec, Ps = sp->prec_sloppy;
     check_prec(Pd);
@@ -330,6 +345,8 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
 // ||bhat - Mhat x|| <= tol ||bhat||, evaluated whenever the iterated normal-equation residual
 // has dropped far enough to make it plausible, and every 50 iterations.
 void cgnr_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *sp, qudax_solve_stats *st) {
+    QX_CHECK(sp->use_schur >= 0 && sp->use_schur <= 2, QUDAX_ERR_ARG, "use_schur must be 0, 1 or 2");
+    SchurForm form_guard(c, sp->use_schur == 2);
     QX_CHECK(c->gauge_loaded, QUDAX_ERR_STATE, "gauge not loaded");
     const int P = sp->prec;
     check_prec(P);

@@ -19,7 +19,7 @@ LIB_PATH = os.environ.get("QUDAX_LIB") or os.path.join(_HERE, "lib", "libqudax.s
 
 HALF, SINGLE, DOUBLE = 2, 4, 8
 EVEN, ODD = 0, 1
-HOP, CLOVER_INV, CLOVER_XPAY = 0, 1, 2
+HOP, CLOVER_INV, CLOVER_XPAY, CLOVER_INV_XPAY = 0, 1, 2, 3
 COMM_NONE, COMM_NCCL, COMM_HOST = 0, 1, 2
 HALO_COMM, HALO_P2P = 0, 1
 PREC_NAMES = {"half": 2, "single": 4, "double": 8, "f16": 2, "f32": 4, "f64": 8}
@@ -124,6 +124,7 @@ SIGNATURES = {
     "qudax_spinor_convert": ([_P, _P, _I, _P, _I], _I),
     "qudax_dslash": ([_P, _P, _P, _P, _I, _I, _I, _I, _D], _I),
     "qudax_matpc": ([_P, _P, _P, _I, _I], _I),
+    "qudax_matpc_sym": ([_P, _P, _P, _I, _I], _I),
     "qudax_dslash_multi": ([_P, ctypes.POINTER(_P), ctypes.POINTER(_P), ctypes.POINTER(_P), _I, _I, _I, _I, _I, _D], _I),
     "qudax_matpc_multi": ([_P, ctypes.POINTER(_P), ctypes.POINTER(_P), _I, _I, _I], _I),
     "qudax_mdagm": ([_P, _P, _P, _I], _I),
@@ -369,6 +370,10 @@ class Context:
     def matpc(self, out, inp, prec, dagger=False):
         self._check(lib().qudax_matpc(self._h, out.data_ptr(), inp.data_ptr(), int(prec), int(bool(dagger))))
 
+    def matpc_sym(self, out, inp, prec, dagger=False):
+        """Symmetric Schur form T_ee^{-1} Mhat (or its explicit adjoint)."""
+        self._check(lib().qudax_matpc_sym(self._h, out.data_ptr(), inp.data_ptr(), int(prec), int(bool(dagger))))
+
     @staticmethod
     def _ptrs(fields):
         return (_P * len(fields))(*[f.data_ptr() for f in fields])
@@ -397,7 +402,9 @@ class Context:
 
     # -- solver
     def _solve_param(self, tol, delta, maxiter, prec, prec_sloppy, use_schur, history=None):
-        sp = SolveParam(float(tol), float(delta), int(maxiter), int(prec_sloppy), int(prec), int(bool(use_schur)))
+        # use_schur: True/1 asymmetric Schur form, 2 (or "sym") symmetric, False/0 even system only
+        us = 2 if use_schur in (2, "sym") else int(bool(use_schur))
+        sp = SolveParam(float(tol), float(delta), int(maxiter), int(prec_sloppy), int(prec), us)
         if history is not None:
             assert history.dtype == np.float64 and history.flags.c_contiguous
             sp.res_history = history.ctypes.data_as(_DP)

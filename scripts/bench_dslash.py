@@ -42,7 +42,7 @@ def main():
         ctx.spinor_load(fi, prec, 1, psi)
         ctx.spinor_load(fx, prec, 0, psi)
         res = {"case": case, "tag": args.tag, "dims": dims}
-        for kind, name in ((0, "hop"), (1, "clover_inv"), (2, "xpay")):
+        for kind, name in ((0, "hop"), (1, "clover_inv"), (2, "xpay"), (3, "inv_xpay")):
             for _ in range(5):
                 ctx.dslash(fo, fi, prec, 0, kind=kind, x=fx, a=-0.1)
             ctx.kernel_timing(True)

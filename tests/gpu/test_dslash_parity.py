@@ -123,6 +123,27 @@ def test_matpc_and_mdagm(torch_cuda, prec, recon):
     ctx.close()
 
 
+@pytest.mark.parametrize("prec,recon", [(8, 18), (4, 12), (2, 12)])
+def test_matpc_sym_and_kernel_kind3(torch_cuda, prec, recon):
+    """Symmetric Schur form and its kernel CLOVER_INV_XPAY
+    (out = x + a T^{-1} D in) against the oracle, both parities and daggers."""
+    case = get_case("8x4x6x8")
+    ctx = make_ctx(case, prec, recon)
+    for p in (0, 1):
+        for dagger in (False, True):
+            got = run_dslash(ctx, case, prec, p, dagger, qudax.CLOVER_INV_XPAY, -0.29)
+            want = oracle.restrict(case.x, p) - 0.29 * case.wc.Tinv_pp(case.wc.Dpq(case.psi, p, dagger), p)
+            assert rel_l2(got, want) <= TOL[prec], (p, dagger)
+    psi_e = oracle.restrict(case.psi, 0)
+    fin, fout = ctx.new_field(prec), ctx.new_field(prec)
+    ctx.spinor_load(fin, prec, 0, case.psi)
+    for dagger in (False, True):
+        ctx.matpc_sym(fout, fin, prec, dagger)
+        got = oracle.restrict(ctx.spinor_store(fout, prec, 0), 0)
+        assert rel_l2(got, case.wc.matpc_sym(psi_e, dagger)) <= TOL[prec], dagger
+    ctx.close()
+
+
 def test_free_field_matpc_closed_form(torch_cuda):
     """Analytic check with no oracle: unit gauge (T = 1), plane wave on even sites."""
     dims = (8, 4, 4, 8)

@@ -114,3 +114,54 @@ def test_cgnr_vs_oracle(torch_cuda, system, prec, recon, tol):
     if prec == 8:
         assert abs(res - st["true_res"]) <= 1e-9
     ctx.close()
+
+
+@pytest.mark.parametrize("mode", [(8, 18, 4, 12, 0.1), (8, 18, 2, 12, 0.1)])
+def test_symmetric_schur_bicgstab_vs_oracle(torch_cuda, system, mode):
+    """use_schur = 2: the symmetric form T_ee^{-1} Mhat.  The solver stops on
+    the symmetric system's true residual; the full-system residual of the reconstructed x is
+    reported and checked by the oracle (it differs from the Schur one by O(|T_ee|))."""
+    U, wc = system
+    prec, recon, ps, rs, delta = mode
+    tol = 1e-12
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=prec, recon=recon, prec_sloppy=ps, recon_sloppy=rs, t_boundary=-1)
+    its = {}
+    for schur in (1, 2):
+        b = qgen.point_source(DIMS, 0, 1)
+        x, st = ctx.solve(b, tol=tol, delta=delta, maxiter=5000, prec=prec, prec_sloppy=ps, use_schur=schur)
+        res_oracle = np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b)
+        print("schur", schur, mode, st["iters"], st["true_res"], res_oracle)
+        assert res_oracle <= 10 * tol
+        assert abs(st["true_res"] - res_oracle) <= 1e-9
+        its[schur] = st["iters"]
+    assert its[2] <= 1.2 * its[1] + 5
+    ctx.close()
+
+
+def test_symmetric_uniform_double_tracks_oracle_history(torch_cuda, system):
+    """delta = 0 fp64 on the symmetric system follows the oracle's BiCGstab on
+    (matpc_sym, prepare_sym) for its first 10 iterations."""
+    U, wc = system
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18)
+    b = qgen.point_source(DIMS, 1, 1)
+    h = np.zeros(200)
+    ctx.solve(b, tol=1e-12, delta=0.0, maxiter=200, prec=8, prec_sloppy=8, history=h, use_schur=2)
+    _, hist = oracle.bicgstab(wc.matpc_sym, wc.prepare_sym(b), tol=1e-12, maxiter=200)
+    hist = np.array(hist)
+    assert np.all(np.abs(h[:10] - hist[:10]) <= 1e-8 * hist[:10])
+    ctx.close()
+
+
+def test_symmetric_cgnr_vs_oracle(torch_cuda, system):
+    U, wc = system
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, t_boundary=-1)
+    b = qgen.point_source(DIMS, 1, 2)
+    x, st = ctx.solve_cgnr(b, tol=1e-12, maxiter=5000, prec=8, use_schur=2)
+    res = np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b)
+    print("cgnr sym", st["iters"], st["true_res"], res)
+    assert res <= 1e-11
+    assert abs(res - st["true_res"]) <= 1e-9
+    ctx.close()
