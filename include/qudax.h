@@ -12,14 +12,19 @@
  * ---------------------------------------------------------------------------------------
  * Conventions (all readings of the paper are listed in DESIGN.md "Readings")
  * ---------------------------------------------------------------------------------------
- * Lattice  global X x Y x Z x T (x fastest, t slowest); partitioned in T only into nranks
- *          equal slabs: rank r owns global t in [r*T_loc,(r+1)*T_loc),
- *          T_loc = T / nranks.  Requires X even, T_loc even (so local and global parity
- *          agree), T_loc >= 2.  Site parity = (x + y + z + t_global) mod 2.
- * Host gauge  const double[4][T_loc][Z][Y][X][3][3][2]: the rank's slab, U_mu(x) stored at x
+ * Lattice  global X x Y x Z x T (x fastest, t slowest), split over a process grid
+ *          Px x Py x Pz x Pt = nranks (the paper splits T only and names
+ *          further dimensions as future work, P:572-578 — SURVEY 8(f) item 4).  Default grid
+ *          (proc_grid all 0): 1 x 1 x 1 x nranks.  Rank r has grid coordinates
+ *          r = ((ct*Pz + cz)*Py + cy)*Px + cx (x fastest) and owns the box
+ *          [c_mu*L_mu, (c_mu+1)*L_mu) with L_mu = dims_mu / P_mu ("local dims").  Requires X_loc
+ *          even and, in every partitioned dimension, an even local extent >= 2 (so local and
+ *          global parity agree); a partitioned X needs Y_loc even too.  Site parity =
+ *          (x + y + z + t) mod 2 in global coordinates.
+ * Host gauge  const double[4][T_loc][Z_loc][Y_loc][X_loc][3][3][2]: the rank's box, U_mu(x) stored at x
  *          (P:425-432), row-major 3x3 complex, mu = 0..3 <-> x, y, z, t.  Borrowed for the
  *          duration of the call only.
- * Host spinor double[T_loc][Z][Y][X][4][3][2] in the DeGrand-Rossi chiral basis (the
+ * Host spinor double[T_loc][Z_loc][Y_loc][X_loc][4][3][2] in the DeGrand-Rossi chiral basis (the
  *          "conventional chiral basis" of eq. (6)).  Borrowed per call.
  * Operator M_kappa = 2 kappa M(eq. (2)) = T - kappa D with T = 1 + 2 kappa A (clover A of
  *          eq. (2); kappa = 1/(2(4+m))).  Even-odd: the solver works
@@ -59,7 +64,7 @@
 extern "C" {
 #endif
 
-#define QUDAX_ABI_VERSION 2
+#define QUDAX_ABI_VERSION 3
 
 typedef enum {
     QUDAX_OK = 0,
@@ -88,10 +93,16 @@ typedef enum { QUDAX_EVEN = 0, QUDAX_ODD = 1 } qudax_parity;
 typedef enum { QUDAX_HOP = 0, QUDAX_CLOVER_INV = 1, QUDAX_CLOVER_XPAY = 2, QUDAX_CLOVER_INV_XPAY = 3 } qudax_dslash_kind;
 
 /* Halo transport:
- *   NONE  nranks must be 1; the Dslash wraps T periodically inside one kernel.
+ *   NONE  nranks must be 1; the Dslash wraps every dimension periodically inside one kernel.
  *   NCCL  ncclSend/ncclRecv of spin-projected faces on a comm stream, overlapped with the
  *         interior kernel; ncclAllReduce for global sums.  With
  *         nranks == 1 this is the loopback test mode (faces go through NCCL to self).
+ *   Faces: T faces carry the 12 reals the diagonal temporal projector keeps, in the storage
+ *         precision (bits only, half with its norm; eq. (6)).  Faces of a partitioned
+ *         X, Y or Z carry the spin-projected half spinor (1 -+ gamma_mu) psi (footnote 3,
+ *         P:665-670), 12 reals in the kernel's arithmetic precision (fp64 for double, fp32 for
+ *         single and half), computed by the pack kernel with the Dslash's own projection code,
+ *         so a partitioned Dslash is bitwise equal to the unpartitioned one.
  *   HOST  faces staged through pinned host memory and exchanged by the caller's hooks
  *         (the paper's non-overlapped strategy); used to run several ranks on
  *         one GPU in tests. */
@@ -110,16 +121,20 @@ typedef enum { QUDAX_COMM_NONE = 0, QUDAX_COMM_NCCL = 1, QUDAX_COMM_HOST = 2 } q
  *         neighbours, because each boundary kernel waits for both of them).  The IPC handles
  *         are swapped once at init over `comm` (host_exchange hook or NCCL); gauge-ghost setup
  *         and global sums keep using `comm`.  With nranks == 1 (comm NONE allowed) the
- *         neighbour is the rank itself: the loopback test of the kernel path. */
+ *         neighbour is the rank itself: the loopback test of the kernel path.  P2P supports a
+ *         T-only split (split_mask = T); other grids return QUDAX_ERR_UNSUPPORTED at init. */
 typedef enum { QUDAX_HALO_COMM = 0, QUDAX_HALO_P2P = 1 } qudax_halo_kind;
 
 typedef struct qudax_ctx qudax_ctx;
 
-/* Host transport hooks for QUDAX_COMM_HOST.  exchange: send send_fwd (bytes) to rank+1 and
- * send_back to rank-1, receive from rank-1 into recv_back and from rank+1 into recv_fwd
- * (periodic ring).  allreduce: in-place sum of n doubles over ranks.  Return 0 on success. */
-typedef int (*qudax_exchange_fn)(const void *send_fwd, const void *send_back, void *recv_back,
-                                 void *recv_fwd, size_t bytes, void *user);
+/* Host transport hooks for QUDAX_COMM_HOST.  exchange: send send_fwd (bytes) to rank_fwd and
+ * send_back to rank_back, receive from rank_back into recv_back and from rank_fwd into recv_fwd
+ * (the two neighbours of this rank along one partitioned dimension; they may be the same rank,
+ * or this rank itself in loopback).  Messages between one pair of ranks must be matched in
+ * call order: send_fwd pairs with the peer's recv_back.  allreduce: in-place sum of n doubles
+ * over ranks.  Return 0 on success. */
+typedef int (*qudax_exchange_fn)(int rank_fwd, int rank_back, const void *send_fwd, const void *send_back,
+                                 void *recv_back, void *recv_fwd, size_t bytes, void *user);
 typedef int (*qudax_allreduce_fn)(double *vals, int n, void *user);
 typedef void *(*qudax_alloc_fn)(size_t bytes, void *user);
 typedef void (*qudax_free_fn)(void *ptr, void *user);
@@ -140,6 +155,12 @@ typedef struct {
     qudax_allreduce_fn host_allreduce;
     void *comm_user;
     int halo;                    /* qudax_halo_kind (0 = COMM) */
+    int proc_grid[4];            /* Px, Py, Pz, Pt with product nranks; all 0 = (1, 1, 1, nranks) */
+    int split_mask;              /* bit mu set: dimension mu uses ghost zones (halo exchange).  0 =
+                                    default: every dimension with P_mu > 1, and T alone when
+                                    nranks == 1 with a transport (loopback).  A non-zero mask must
+                                    contain every dimension with P_mu > 1; extra bits are loopback
+                                    dimensions (the rank is its own neighbour) for tests. */
 } qudax_init_param;
 
 typedef struct {
@@ -181,12 +202,19 @@ typedef struct {
 } qudax_site_model;
 
 typedef struct {
-    int T_loc, t0;               /* local extent and first global timeslice */
-    int rank_fwd, rank_back;     /* T-ring neighbours */
-    long V_loc, V_h, V_s, face_sites; /* local volume, per-parity volume, XYZ, XYZ/2 */
+    int T_loc, t0;               /* local T extent and first global timeslice */
+    int rank_fwd, rank_back;     /* T-direction neighbours */
+    long V_loc, V_h, V_s, face_sites; /* local volume, per-parity volume, X_loc*Y_loc*Z_loc, V_s/2 */
     int applies_bc_fwd, applies_bc_back; /* this rank owns global t=T-1 / t=0 */
-    size_t face_bytes[3];        /* one projected face (12 reals per site) in half/single/double,
+    size_t face_bytes[3];        /* one T face (12 reals per site) in half/single/double,
                                     half including its per-site norms */
+    int proc_grid[4];            /* process grid */
+    int coords[4];               /* this rank's grid coordinates */
+    int local_dims[4];           /* X_loc, Y_loc, Z_loc, T_loc */
+    int origin[4];               /* global coordinates of local site (0,0,0,0) */
+    int nb_fwd[4], nb_back[4];   /* neighbour ranks along each dimension (self if P_mu = 1) */
+    int split_mask;              /* dimensions with ghost zones (see qudax_init_param) */
+    long face_sites_dim[4];      /* per-parity face sites V_loc / L_mu / 2 along each dimension */
 } qudax_partition;
 
 /* Accumulated CUDA-event timing of the Dslash kernel launches since qudax_kernel_timing(ctx, 1). */
@@ -202,8 +230,10 @@ typedef struct {
 /* ---- host-only helpers (no GPU needed) ---- */
 int qudax_abi_version(void);
 const char *qudax_status_string(int status);
-/* Partition bookkeeping of rank `rank` of `nranks`. */
-qudax_status qudax_partition_info(const int global_dims[4], int nranks, int rank, qudax_partition *out);
+/* Partition bookkeeping of rank `rank` of `nranks`.  proc_grid may be
+ * NULL (T only); split_mask as in qudax_init_param (0 = default). */
+qudax_status qudax_partition_info(const int global_dims[4], const int proc_grid[4], int nranks, int rank,
+                                  int split_mask, qudax_partition *out);
 /* Site model for one Dslash kernel of `kind` (flops: 1320 + 504 clover + 48 xpay, Q16), or for
  * the whole Mhat when kind = -1 (3696 flops / 2976 bytes at fp32 recon 12), or for
  * the single-launch (fused) Mhat when kind = -2 (compulsory bytes: links once, T and T^{-1},
@@ -226,8 +256,9 @@ qudax_status qudax_kernel_timing(qudax_ctx *ctx, int enable);
 qudax_status qudax_get_kernel_stats(qudax_ctx *ctx, int prec_filter, qudax_kernel_stats *out);
 
 /* ---- gauge field and clover (setup) ----
- * Uploads the host slab, exchanges the gauge ghost / clover halo timeslices with the T
- * neighbours (once), builds A and T^{-1} in fp64 on the device and stores gauge + clover in
+ * Uploads the host box, exchanges a one-site gauge halo (with corners: one dimension after the
+ * other, each message including the halos already received) with the neighbours of every
+ * partitioned dimension (once), builds A and T^{-1} in fp64 on the device and stores gauge + clover in
  * the outer and sloppy (precision, reconstruct) formats.  Returns QUDAX_ERR_UNSUPPORTED for
  * reconstruct 8 when some link has |u01|^2 + |u02|^2 < 1e-6. */
 qudax_status qudax_gauge_load(qudax_ctx *ctx, const double *host_gauge, const qudax_gauge_param *p);

@@ -47,6 +47,13 @@ void *halloc(qudax_ctx *c, size_t bytes) {
     return p;
 }
 
+static void hfree(qudax_ctx *c, void *p) {
+    if (!p) return;
+    auto it = std::find(c->host_allocs.begin(), c->host_allocs.end(), p);
+    if (it != c->host_allocs.end()) c->host_allocs.erase(it);
+    cudaFreeHost(p);
+}
+
 static void dfree(qudax_ctx *c, void *p) {
     if (!p) return;
     auto it = std::find(c->allocs.begin(), c->allocs.end(), p);
@@ -69,49 +76,95 @@ static qudax_ctx::GaugeCopy &gauge_for(qudax_ctx *c, int prec) {
 static qudax_ctx::Halo &halo_for(qudax_ctx *c, int prec) {
     auto &h = c->halo[prec_idx(prec)];
     if (!h.valid) {
-        h.bytes = face_bytes(prec, c->g.fstride);
-        h.sb = dalloc(c, h.bytes);
-        h.sf = dalloc(c, h.bytes);
-        h.gb = dalloc(c, h.bytes);
-        h.gf = dalloc(c, h.bytes);
-        if (c->comm == QUDAX_COMM_HOST) {
-            h.h_sb = halloc(c, h.bytes);
-            h.h_sf = halloc(c, h.bytes);
-            h.h_gb = halloc(c, h.bytes);
-            h.h_gf = halloc(c, h.bytes);
+        const Geom &g = c->g;
+        const bool host = c->comm == QUDAX_COMM_HOST;
+        if (g.split & 8) {
+            h.bytes = face_bytes(prec, g.fstride);
+            h.sb = dalloc(c, h.bytes);
+            h.sf = dalloc(c, h.bytes);
+            h.gb = dalloc(c, h.bytes);
+            h.gf = dalloc(c, h.bytes);
+            if (host) {
+                h.h_sb = halloc(c, h.bytes);
+                h.h_sf = halloc(c, h.bytes);
+                h.h_gb = halloc(c, h.bytes);
+                h.h_gf = halloc(c, h.bytes);
+            }
+        }
+        for (int m = 0; m < 3; ++m) {
+            if (!(g.split >> m & 1)) continue;
+            const size_t b = sface_bytes(prec, g.fsd[m]);
+            h.sbytes[m] = b;
+            h.ssb[m] = dalloc(c, b);
+            h.ssf[m] = dalloc(c, b);
+            h.sgb[m] = dalloc(c, b);
+            h.sgf[m] = dalloc(c, b);
+            if (host) {
+                h.h_ssb[m] = halloc(c, b);
+                h.h_ssf[m] = halloc(c, b);
+                h.h_sgb[m] = halloc(c, b);
+                h.h_sgf[m] = halloc(c, b);
+            }
         }
         h.valid = true;
     }
     return h;
 }
 
-static inline int rank_fwd(const Geom &g) { return (g.rank + 1) % g.nranks; }
-static inline int rank_back(const Geom &g) { return (g.rank - 1 + g.nranks) % g.nranks; }
+static inline int rank_fwd(const Geom &g) { return g.nbf[3]; }
+static inline int rank_back(const Geom &g) { return g.nbb[3]; }
 
-// Exchange of two device buffers of `bytes` with the T neighbours: send_fwd -> rank+1,
-// send_back -> rank-1, recv_back <- rank-1, recv_fwd <- rank+1.  On NCCL it is enqueued on
-// `s`; on HOST it is staged through pinned memory and completes before return.
-static void exchange(qudax_ctx *c, const void *send_fwd, const void *send_back, void *recv_back, void *recv_fwd,
-                     size_t bytes, cudaStream_t s, void *h_sf, void *h_sb, void *h_gb, void *h_gf) {
+// One neighbour exchange along dimension mu: send_fwd -> nbf[mu], send_back -> nbb[mu],
+// recv_back <- nbb[mu], recv_fwd <- nbf[mu].
+struct Xfer {
+    int mu;
+    const void *send_fwd, *send_back;
+    void *recv_back, *recv_fwd;
+    size_t bytes;
+    void *h_sf, *h_sb, *h_gb, *h_gf;  // pinned staging (HOST)
+};
+// All transfers of one halo: on NCCL one group enqueued on `s` (the messages of different
+// dimensions go to different peers, so their order within the group is free); on HOST staged
+// through pinned memory, one hook call per dimension, complete before return.  A dimension whose
+// neighbour is this rank (loopback on HOST) is a device copy.
+static void exchange_all(qudax_ctx *c, const Xfer *x, int n, cudaStream_t s) {
     const Geom &g = c->g;
     if (c->comm == QUDAX_COMM_NCCL) {
         QX_NCCL(ncclGroupStart());
-        QX_NCCL(ncclSend(send_fwd, bytes, ncclChar, rank_fwd(g), c->nccl, s));
-        QX_NCCL(ncclRecv(recv_back, bytes, ncclChar, rank_back(g), c->nccl, s));
-        QX_NCCL(ncclSend(send_back, bytes, ncclChar, rank_back(g), c->nccl, s));
-        QX_NCCL(ncclRecv(recv_fwd, bytes, ncclChar, rank_fwd(g), c->nccl, s));
+        for (int k = 0; k < n; ++k) {
+            const int f = g.nbf[x[k].mu], b = g.nbb[x[k].mu];
+            QX_NCCL(ncclSend(x[k].send_fwd, x[k].bytes, ncclChar, f, c->nccl, s));
+            QX_NCCL(ncclRecv(x[k].recv_back, x[k].bytes, ncclChar, b, c->nccl, s));
+            QX_NCCL(ncclSend(x[k].send_back, x[k].bytes, ncclChar, b, c->nccl, s));
+            QX_NCCL(ncclRecv(x[k].recv_fwd, x[k].bytes, ncclChar, f, c->nccl, s));
+        }
         QX_NCCL(ncclGroupEnd());
     } else if (c->comm == QUDAX_COMM_HOST) {
-        QX_CUDA(cudaMemcpyAsync(h_sf, send_fwd, bytes, cudaMemcpyDeviceToHost, s));
-        QX_CUDA(cudaMemcpyAsync(h_sb, send_back, bytes, cudaMemcpyDeviceToHost, s));
-        QX_CUDA(cudaStreamSynchronize(s));
-        int rc = c->host_exchange(h_sf, h_sb, h_gb, h_gf, bytes, c->comm_user);
-        if (rc) throw Error(QUDAX_ERR_COMM, "host_exchange hook failed");
-        QX_CUDA(cudaMemcpyAsync(recv_back, h_gb, bytes, cudaMemcpyHostToDevice, s));
-        QX_CUDA(cudaMemcpyAsync(recv_fwd, h_gf, bytes, cudaMemcpyHostToDevice, s));
+        for (int k = 0; k < n; ++k) {
+            const Xfer &t = x[k];
+            const int f = g.nbf[t.mu], b = g.nbb[t.mu];
+            if (f == g.rank && b == g.rank) {
+                QX_CUDA(cudaMemcpyAsync(t.recv_back, t.send_fwd, t.bytes, cudaMemcpyDeviceToDevice, s));
+                QX_CUDA(cudaMemcpyAsync(t.recv_fwd, t.send_back, t.bytes, cudaMemcpyDeviceToDevice, s));
+                continue;
+            }
+            QX_CUDA(cudaMemcpyAsync(t.h_sf, t.send_fwd, t.bytes, cudaMemcpyDeviceToHost, s));
+            QX_CUDA(cudaMemcpyAsync(t.h_sb, t.send_back, t.bytes, cudaMemcpyDeviceToHost, s));
+            QX_CUDA(cudaStreamSynchronize(s));
+            int rc = c->host_exchange(f, b, t.h_sf, t.h_sb, t.h_gb, t.h_gf, t.bytes, c->comm_user);
+            if (rc) throw Error(QUDAX_ERR_COMM, "host_exchange hook failed");
+            QX_CUDA(cudaMemcpyAsync(t.recv_back, t.h_gb, t.bytes, cudaMemcpyHostToDevice, s));
+            QX_CUDA(cudaMemcpyAsync(t.recv_fwd, t.h_gf, t.bytes, cudaMemcpyHostToDevice, s));
+        }
     } else {
         throw Error(QUDAX_ERR_STATE, "exchange without a transport");
     }
+}
+// T-direction exchange of two device buffers (gauge-free helper used by setup code)
+static void exchange(qudax_ctx *c, const void *send_fwd, const void *send_back, void *recv_back, void *recv_fwd,
+                     size_t bytes, cudaStream_t s, void *h_sf, void *h_sb, void *h_gb, void *h_gf) {
+    Xfer x{3, send_fwd, send_back, recv_back, recv_fwd, bytes, h_sf, h_sb, h_gb, h_gf};
+    exchange_all(c, &x, 1, s);
 }
 
 static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res);
@@ -210,14 +263,25 @@ static DslashArgs base_args(qudax_ctx *c, const qudax_ctx::GaugeCopy &gc, int pr
     args.Vh = (int)g.Vh; args.F = (int)g.F;
     args.stride = g.stride; args.fstride = g.fstride;
     args.parity = p;
-    args.bc_fwd = (g.rank == g.nranks - 1) ? (double)c->t_bc : 1.0;
-    args.bc_back = (g.rank == 0) ? (double)c->t_bc : 1.0;
+    // the antiperiodic sign belongs to the hops that cross global t = T-1 <-> 0 (reading Q5)
+    args.bc_fwd = (g.c[3] == g.P[3] - 1) ? (double)c->t_bc : 1.0;
+    args.bc_back = (g.c[3] == 0) ? (double)c->t_bc : 1.0;
     args.a = a;
     args.reverse = reverse;
     args.nrhs = 1;
     for (int m = 0; m < 4; ++m)
         for (int q = 0; q < 2; ++q) args.gauge[m][q] = gc.d[m][q];
-    args.gauge_ghost = gc.ghost[1 - p];
+    args.gauge_ghost = gc.ghost[3][1 - p];
+    args.smask = spatial_split(g);
+    for (int m = 0; m < 3; ++m) {
+        args.sfs[m] = g.fsd[m];
+        args.gauge_sghost[m] = gc.ghost[m][1 - p];
+    }
+    for (int m = 0; m < 4; ++m) {
+        args.blo[m] = g.blo[m];
+        args.bn[m] = g.bn[m];
+    }
+    args.blist = c->blist;
     if (kind != QUDAX_HOP) {
         auto &cl = c->clov[prec_idx(prec)];
         QX_CHECK(cl.valid, QUDAX_ERR_STATE, "no clover in this precision");
@@ -238,7 +302,8 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     DslashArgs args = base_args(c, gc, prec, p, kind, a, reverse);
     args.in = in; args.out = out; args.x = x;
     int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
-    const bool split = c->comm == QUDAX_COMM_NCCL && !c->p2p.on && c->overlap && g.T_loc > 2;
+    const long n_int = g.n_int, n_bnd = g.Vh - g.n_int;
+    const bool split = c->comm == QUDAX_COMM_NCCL && !c->p2p.on && c->overlap && n_int > 0;
     const bool multi = (g.nranks > 1);  // cross-rank sums needed before the scalar recurrence
     if (red) {
         QX_CHECK(red->kind != RED_XDOT_NORM || kind >= QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
@@ -247,11 +312,10 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / 32) + 64)));
         args.red_kind = red->kind;
         args.rhat = red->rhat;
-        const int ni = (int)((g.T_loc - 2) * g.F), nb = (int)(2 * g.F);
         args.tail.partials = c->dpart;
         args.tail.counter = c->d_counter;
-        args.tail.total_blocks = split ? dslash_blocks_any(prec, gc.recon, dagger, kind, ni) +
-                                             dslash_blocks_any(prec, gc.recon, dagger, kind, nb)
+        args.tail.total_blocks = split ? dslash_blocks_any(prec, gc.recon, dagger, kind, (int)n_int) +
+                                             dslash_blocks_any(prec, gc.recon, dagger, kind, (int)n_bnd)
                                        : dslash_blocks_any(prec, gc.recon, dagger, kind, (int)g.Vh);
         args.tail.out = red->S ? red->S->red : c->red_out;
         args.tail.S = red->S;
@@ -270,7 +334,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         if (!red->S) global_sum(c, c->red_out, 3, red->res);
         else if (multi) device_sum_coef(c, red->S->red, 3, red->S, red->coef_mode);
     };
-    if (c->p2p.on) {  // kernel-initiated halo over peer memory (QUDAX_HALO_P2P)
+    if (c->p2p.on) {  // kernel-initiated halo over peer memory (QUDAX_HALO_P2P), T-only split
         auto &q = c->p2p;
         const int pi = prec_idx(prec);
         args.ghosted = 1;
@@ -309,36 +373,53 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         finish_red();
         return;
     }
-    if (c->comm == QUDAX_COMM_NONE) {
+    if (c->comm == QUDAX_COMM_NONE || g.split == 0) {
         args.ghosted = 0;
         launch(RANGE_ALL, (int)g.Vh);
         finish_red();
         return;
     }
     auto &h = halo_for(c, prec);
-    args.ghosted = 1;
+    args.ghosted = (g.split >> 3) & 1;
     args.ghost_back = h.gb;
     args.ghost_fwd = h.gf;
+    Xfer xf[4];
+    int nx = 0;
+    for (int m = 0; m < 3; ++m) {
+        args.sghost_back[m] = h.sgb[m];
+        args.sghost_fwd[m] = h.sgf[m];
+        if (g.split >> m & 1)
+            xf[nx++] = Xfer{m, h.ssf[m], h.ssb[m], h.sgb[m], h.sgf[m], h.sbytes[m], h.h_ssf[m], h.h_ssb[m], h.h_sgb[m], h.h_sgf[m]};
+    }
+    if (g.split & 8) xf[nx++] = Xfer{3, h.sf, h.sb, h.gb, h.gf, h.bytes, h.h_sf, h.h_sb, h.h_gb, h.h_gf};
+    auto pack_all = [&](cudaStream_t st) {
+        if (g.split & 8) {
+            launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, st);
+            c->launches += 1;
+        }
+        if (spatial_split(g)) {
+            launch_pack_spatial(prec, dagger, g, 1 - p, in, h.ssb, h.ssf, st);
+            c->launches += 1;
+        }
+    };
     if (c->comm == QUDAX_COMM_NCCL) {
         // comm stream: wait for `in` (and for the previous boundary kernel, which read the ghosts)
         QX_CUDA(cudaEventRecord(c->ev_in, c->stream));
         QX_CUDA(cudaStreamWaitEvent(c->comm_stream, c->ev_in, 0));
-        launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, c->comm_stream);
-        exchange(c, h.sf, h.sb, h.gb, h.gf, h.bytes, c->comm_stream, nullptr, nullptr, nullptr, nullptr);
+        pack_all(c->comm_stream);
+        exchange_all(c, xf, nx, c->comm_stream);
         QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
-        c->launches += 1;
         if (split) {
-            launch(RANGE_INTERIOR, (int)((g.T_loc - 2) * g.F));
+            launch(RANGE_INTERIOR, (int)n_int);
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
-            launch(RANGE_BOUNDARY, (int)(2 * g.F));
+            launch(RANGE_BOUNDARY, (int)n_bnd);
         } else {
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
             launch(RANGE_ALL, (int)g.Vh);
         }
     } else {  // HOST: paper strategy 1 (no overlap)
-        launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, c->stream);
-        exchange(c, h.sf, h.sb, h.gb, h.gf, h.bytes, c->stream, h.h_sf, h.h_sb, h.h_gb, h.h_gf);
-        c->launches += 1;
+        pack_all(c->stream);
+        exchange_all(c, xf, nx, c->stream);
         launch(RANGE_ALL, (int)g.Vh);
     }
     finish_red();
@@ -601,9 +682,10 @@ static void gauge_load(qudax_ctx *c, const double *host, const qudax_gauge_param
     // drop a previous configuration's copies (fields of the previous load are released)
     for (int k = 0; k < c->ncopies; ++k) {
         for (int m = 0; m < 4; ++m)
-            for (int q = 0; q < 2; ++q) dfree(c, c->gcopy[k].d[m][q]);
-        dfree(c, c->gcopy[k].ghost[0]);
-        dfree(c, c->gcopy[k].ghost[1]);
+            for (int q = 0; q < 2; ++q) {
+                dfree(c, c->gcopy[k].d[m][q]);
+                dfree(c, c->gcopy[k].ghost[m][q]);
+            }
         c->gcopy[k] = qudax_ctx::GaugeCopy{};
     }
     for (auto &cl : c->clov) {
@@ -617,26 +699,43 @@ static void gauge_load(qudax_ctx *c, const double *host, const qudax_gauge_param
     c->csw = p->csw;
     c->t_bc = p->t_boundary;
 
-    // 1. upload the slab into the extended fp64 buffer [T_loc+2][4][Vs][18]
-    const size_t link_d = 18;
-    const size_t slice = (size_t)4 * g.Vs * link_d;  // doubles per extended timeslice
-    double *ext = static_cast<double *>(dalloc(c, sizeof(double) * slice * (g.T_loc + 2)));
-    for (int mu = 0; mu < 4; ++mu) {
-        QX_CUDA(cudaMemcpy2DAsync(ext + slice + (size_t)mu * g.Vs * link_d, sizeof(double) * slice,
-                                  host + (size_t)mu * g.T_loc * g.Vs * link_d, sizeof(double) * g.Vs * link_d,
-                                  sizeof(double) * g.Vs * link_d, g.T_loc, cudaMemcpyHostToDevice, c->stream));
+    // 1. upload the box and scatter it into the extended site-major fp64 buffer
+    //    ext[Et][Ez][Ey][Ex][4][18] (one-site halo on every split dimension)
+    double *ext = static_cast<double *>(dalloc(c, sizeof(double) * 72 * ext_sites(g)));
+    {
+        double *box = static_cast<double *>(dalloc(c, sizeof(double) * 72 * g.V));
+        QX_CUDA(cudaMemcpyAsync(box, host, sizeof(double) * 72 * g.V, cudaMemcpyHostToDevice, c->stream));
+        launch_ext_fill(g, box, ext, c->stream);
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        dfree(c, box);
     }
-    // 2. gauge ghost + clover halo: one full timeslice from each T neighbour, once
-    double *first = ext + slice, *last = ext + slice * g.T_loc;
-    double *halo_back = ext, *halo_fwd = ext + slice * (g.T_loc + 1);
-    if (c->comm == QUDAX_COMM_NONE || g.nranks == 1) {
-        QX_CUDA(cudaMemcpyAsync(halo_back, last, sizeof(double) * slice, cudaMemcpyDeviceToDevice, c->stream));
-        QX_CUDA(cudaMemcpyAsync(halo_fwd, first, sizeof(double) * slice, cudaMemcpyDeviceToDevice, c->stream));
-    } else {
-        void *hs[4] = {nullptr, nullptr, nullptr, nullptr};
-        if (c->comm == QUDAX_COMM_HOST)
-            for (auto &q : hs) q = halloc(c, sizeof(double) * slice);
-        exchange(c, last, first, halo_back, halo_fwd, sizeof(double) * slice, c->stream, hs[0], hs[1], hs[2], hs[3]);
+    // 2. gauge ghost + clover halo: along each split dimension in turn, the first and
+    //    last interior cross-sections (with the halos already received: corners) go to the
+    //    neighbours and come back as the two halo cross-sections.  Once per configuration.
+    for (int mu = 0; mu < 4; ++mu) {
+        if (!(g.split >> mu & 1)) continue;
+        const long n = ext_slice_doubles(g, mu);
+        const size_t bytes = sizeof(double) * n;
+        double *buf = static_cast<double *>(dalloc(c, 4 * bytes));
+        double *s_lo = buf, *s_hi = buf + n, *r_lo = buf + 2 * n, *r_hi = buf + 3 * n;
+        launch_ext_slice(g, ext, mu, 1, s_lo, true, c->stream);             // local x_mu = 0
+        launch_ext_slice(g, ext, mu, g.L[mu], s_hi, true, c->stream);       // local x_mu = L-1
+        if (c->comm == QUDAX_COMM_NONE || (g.nbf[mu] == g.rank && g.nbb[mu] == g.rank)) {
+            QX_CUDA(cudaMemcpyAsync(r_lo, s_hi, bytes, cudaMemcpyDeviceToDevice, c->stream));
+            QX_CUDA(cudaMemcpyAsync(r_hi, s_lo, bytes, cudaMemcpyDeviceToDevice, c->stream));
+        } else {
+            void *hs[4] = {nullptr, nullptr, nullptr, nullptr};
+            if (c->comm == QUDAX_COMM_HOST)
+                for (auto &q : hs) q = halloc(c, bytes);
+            Xfer x{mu, s_hi, s_lo, r_lo, r_hi, bytes, hs[0], hs[1], hs[2], hs[3]};
+            exchange_all(c, &x, 1, c->stream);
+            QX_CUDA(cudaStreamSynchronize(c->stream));
+            for (auto &q : hs) hfree(c, q);
+        }
+        launch_ext_slice(g, ext, mu, 0, r_lo, false, c->stream);            // local x_mu = -1
+        launch_ext_slice(g, ext, mu, g.L[mu] + 1, r_hi, false, c->stream);  // local x_mu = L
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        dfree(c, buf);
     }
     // 3. pack each (precision, reconstruct) copy
     int *bad = c->d_flag;
@@ -650,7 +749,9 @@ static void gauge_load(qudax_ctx *c, const double *host, const qudax_gauge_param
         const size_t b = soa_bytes(pr, rc, g.stride);
         for (int m = 0; m < 4; ++m)
             for (int q = 0; q < 2; ++q) gc.d[m][q] = dalloc(c, b);
-        for (int q = 0; q < 2; ++q) gc.ghost[q] = dalloc(c, soa_bytes(pr, rc, g.fstride));
+        for (int m = 0; m < 4; ++m)
+            if (g.split >> m & 1)
+                for (int q = 0; q < 2; ++q) gc.ghost[m][q] = dalloc(c, soa_bytes(pr, rc, g.fsd[m]));
         launch_gauge_pack2(pr, rc, g, ext, gc.d, gc.ghost, bad, c->stream);
         c->launches += 1;
     }
@@ -718,28 +819,72 @@ qudax_status guard(qudax_ctx *c, F &&fn) {
     }
 }
 
-qudax_status fill_partition(const int gd[4], int nranks, int rank, qudax_partition *o) {
+// Process-grid bookkeeping (multi-dimensional split: SURVEY 8(f) item 4).
+// halo_p2p: the init's halo kind (a P2P halo at one rank defaults to a T loopback).
+qudax_status fill_partition(const int gd[4], const int grid_in[4], int nranks, int rank, int split_mask, int comm,
+                            int halo_p2p, qudax_partition *o) {
     if (!gd || !o || nranks < 1 || rank < 0 || rank >= nranks) return QUDAX_ERR_ARG;
+    int P[4] = {1, 1, 1, nranks};
+    if (grid_in && (grid_in[0] | grid_in[1] | grid_in[2] | grid_in[3])) {
+        for (int k = 0; k < 4; ++k) P[k] = grid_in[k];
+    }
+    long prod = 1;
+    for (int k = 0; k < 4; ++k) {
+        if (gd[k] < 1 || P[k] < 1 || gd[k] % P[k]) return QUDAX_ERR_ARG;
+        prod *= P[k];
+    }
+    if (prod != nranks) return QUDAX_ERR_ARG;
+    int L[4], c[4];
+    for (int k = 0; k < 4; ++k) L[k] = gd[k] / P[k];
+    {
+        int r = rank;
+        for (int k = 0; k < 4; ++k) {
+            c[k] = r % P[k];
+            r /= P[k];
+        }
+    }
+    int split = 0;
     for (int k = 0; k < 4; ++k)
-        if (gd[k] < 1) return QUDAX_ERR_ARG;
-    if (gd[0] % 2) return QUDAX_ERR_ARG;
-    if (gd[3] % nranks) return QUDAX_ERR_ARG;
-    const int T_loc = gd[3] / nranks;
-    if (T_loc < 2 || T_loc % 2) return QUDAX_ERR_ARG;
+        if (P[k] > 1) split |= 1 << k;
+    if (split_mask) {
+        if ((split_mask & split) != split || (split_mask & ~15)) return QUDAX_ERR_ARG;
+        split = split_mask;
+    } else if (split == 0 && (comm != QUDAX_COMM_NONE || halo_p2p)) {
+        split = 8;  // one rank with a transport: T loopback (the split path at N = 1)
+    }
+    if (L[0] % 2) return QUDAX_ERR_ARG;
+    if (L[3] < 2 || L[3] % 2) return QUDAX_ERR_ARG;
+    for (int k = 0; k < 4; ++k)
+        if ((split >> k & 1) && (L[k] < 2 || L[k] % 2)) return QUDAX_ERR_ARG;
+    if ((split & 1) && L[1] % 2) return QUDAX_ERR_ARG;  // X faces pair their sites along y
     std::memset(o, 0, sizeof(*o));
-    o->T_loc = T_loc;
-    o->t0 = rank * T_loc;
-    o->rank_fwd = (rank + 1) % nranks;
-    o->rank_back = (rank - 1 + nranks) % nranks;
-    o->V_s = (long)gd[0] * gd[1] * gd[2];
-    o->V_loc = o->V_s * T_loc;
+    o->T_loc = L[3];
+    o->t0 = c[3] * L[3];
+    o->V_s = (long)L[0] * L[1] * L[2];
+    o->V_loc = o->V_s * L[3];
     o->V_h = o->V_loc / 2;
     o->face_sites = o->V_s / 2;
-    o->applies_bc_fwd = (rank == nranks - 1);
-    o->applies_bc_back = (rank == 0);
+    o->applies_bc_fwd = (c[3] == P[3] - 1);
+    o->applies_bc_back = (c[3] == 0);
     o->face_bytes[0] = (size_t)o->face_sites * (12 * 2 + 4);
     o->face_bytes[1] = (size_t)o->face_sites * 12 * 4;
     o->face_bytes[2] = (size_t)o->face_sites * 12 * 8;
+    auto rank_of = [&](const int cc[4]) { return ((cc[3] * P[2] + cc[2]) * P[1] + cc[1]) * P[0] + cc[0]; };
+    for (int k = 0; k < 4; ++k) {
+        o->proc_grid[k] = P[k];
+        o->coords[k] = c[k];
+        o->local_dims[k] = L[k];
+        o->origin[k] = c[k] * L[k];
+        int cf[4] = {c[0], c[1], c[2], c[3]}, cb[4] = {c[0], c[1], c[2], c[3]};
+        cf[k] = (c[k] + 1) % P[k];
+        cb[k] = (c[k] - 1 + P[k]) % P[k];
+        o->nb_fwd[k] = rank_of(cf);
+        o->nb_back[k] = rank_of(cb);
+        o->face_sites_dim[k] = o->V_loc / L[k] / 2;
+    }
+    o->rank_fwd = o->nb_fwd[3];
+    o->rank_back = o->nb_back[3];
+    o->split_mask = split;
     return QUDAX_OK;
 }
 }  // namespace
@@ -763,8 +908,9 @@ const char *qudax_status_string(int s) {
     }
 }
 
-qudax_status qudax_partition_info(const int global_dims[4], int nranks, int rank, qudax_partition *out) {
-    return fill_partition(global_dims, nranks, rank, out);
+qudax_status qudax_partition_info(const int global_dims[4], const int proc_grid[4], int nranks, int rank,
+                                  int split_mask, qudax_partition *out) {
+    return fill_partition(global_dims, proc_grid, nranks, rank, split_mask, QUDAX_COMM_NONE, 0, out);
 }
 
 qudax_status qudax_model(int prec, int recon, int kind, qudax_site_model *o) {
@@ -844,7 +990,7 @@ static void setup_p2p(qudax_ctx *c) {
     QX_CUDA(cudaIpcGetMemHandle(&mine, q.base));
     if (c->comm == QUDAX_COMM_HOST) {
         cudaIpcMemHandle_t s0 = mine, s1 = mine;
-        if (c->host_exchange(&s0, &s1, &hb, &hf, sizeof(mine), c->comm_user))
+        if (c->host_exchange(g.nbf[3], g.nbb[3], &s0, &s1, &hb, &hf, sizeof(mine), c->comm_user))
             throw Error(QUDAX_ERR_COMM, "host_exchange hook failed (IPC handles)");
     } else if (c->comm == QUDAX_COMM_NCCL) {
         char *d = static_cast<char *>(dalloc(c, 3 * sizeof(mine)));
@@ -873,23 +1019,53 @@ static void setup_p2p(qudax_ctx *c) {
 qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
     if (!out || !p) return QUDAX_ERR_ARG;
     *out = nullptr;
+    if (p->comm < 0 || p->comm > 2) return QUDAX_ERR_ARG;
+    if (p->halo != QUDAX_HALO_COMM && p->halo != QUDAX_HALO_P2P) return QUDAX_ERR_ARG;
     qudax_partition part;
-    if (fill_partition(p->global_dims, p->nranks, p->rank, &part) != QUDAX_OK) return QUDAX_ERR_ARG;
+    if (fill_partition(p->global_dims, p->proc_grid, p->nranks, p->rank, p->split_mask, p->comm,
+                       p->halo == QUDAX_HALO_P2P, &part) != QUDAX_OK)
+        return QUDAX_ERR_ARG;
     if (p->comm == QUDAX_COMM_NONE && p->nranks != 1) return QUDAX_ERR_ARG;
     if (p->comm == QUDAX_COMM_NCCL && !p->nccl_id) return QUDAX_ERR_ARG;
     if (p->comm == QUDAX_COMM_HOST && (!p->host_exchange || !p->host_allreduce)) return QUDAX_ERR_ARG;
-    if (p->comm < 0 || p->comm > 2) return QUDAX_ERR_ARG;
-    if (p->halo != QUDAX_HALO_COMM && p->halo != QUDAX_HALO_P2P) return QUDAX_ERR_ARG;
+    // the kernel-initiated halo covers the T faces; the comm halo every dimension
+    if (p->halo == QUDAX_HALO_P2P && part.split_mask != 8) return QUDAX_ERR_UNSUPPORTED;
+    // a loopback dimension without a transport has nobody to move its faces
+    if (p->comm == QUDAX_COMM_NONE && p->halo != QUDAX_HALO_P2P && part.split_mask) return QUDAX_ERR_ARG;
     auto *c = new qudax_ctx();
     qudax_status st = guard(c, [&] {
         Geom &g = c->g;
-        g.X = p->global_dims[0]; g.Y = p->global_dims[1]; g.Z = p->global_dims[2]; g.T = p->global_dims[3];
+        for (int k = 0; k < 4; ++k) {
+            g.G[k] = p->global_dims[k];
+            g.L[k] = part.local_dims[k];
+            g.P[k] = part.proc_grid[k];
+            g.c[k] = part.coords[k];
+            g.o[k] = part.origin[k];
+            g.nbf[k] = part.nb_fwd[k];
+            g.nbb[k] = part.nb_back[k];
+            g.Fd[k] = part.face_sites_dim[k];
+            g.fsd[k] = pad64(g.Fd[k]);
+        }
+        g.split = part.split_mask;
+        g.X = g.L[0]; g.Y = g.L[1]; g.Z = g.L[2]; g.T = p->global_dims[3];
         g.nranks = p->nranks; g.rank = p->rank;
         g.T_loc = part.T_loc; g.t0 = part.t0;
         g.Xh = g.X / 2;
         g.Vs = part.V_s; g.V = part.V_loc; g.Vh = part.V_h; g.F = part.face_sites;
         g.stride = pad64(g.Vh);
         g.fstride = pad64(g.F);
+        // interior box in (xh, y, z, t): one site off every split face (a split X drops the
+        // first and last xh of each row, which holds x = 0 or x = X-1)
+        {
+            const int ext[4] = {g.Xh, g.Y, g.Z, g.T_loc};
+            g.n_int = 1;
+            for (int k = 0; k < 4; ++k) {
+                const int s = (g.split >> k) & 1;
+                g.blo[k] = s;
+                g.bn[k] = std::max(0, ext[k] - 2 * s);
+                g.n_int *= g.bn[k];
+            }
+        }
         QX_CHECK(g.V < (1L << 30), QUDAX_ERR_ARG, "local volume too large for 32-bit site indexing");
         c->device = p->device;
         if (const char *ng = std::getenv("QUDAX_NO_GRAPHS")) c->no_graphs = (ng[0] == '1');
@@ -928,6 +1104,26 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         if (p->halo == QUDAX_HALO_P2P) {
             setup_p2p(c);
             c->p2p.on = true;
+        }
+        if (spatial_split(g)) {  // boundary sites of a multi-dimensional split: the box complement
+            std::vector<int> bl;
+            bl.reserve((size_t)(g.Vh - g.n_int));
+            for (long i = 0; i < g.Vh; ++i) {
+                long r = i;
+                const int xh = (int)(r % g.Xh);
+                r /= g.Xh;
+                const int y = (int)(r % g.Y);
+                r /= g.Y;
+                const int z = (int)(r % g.Z);
+                const int t = (int)(r / g.Z);
+                const int cc[4] = {xh, y, z, t};
+                bool in = true;
+                for (int k = 0; k < 4; ++k) in &= cc[k] >= g.blo[k] && cc[k] < g.blo[k] + g.bn[k];
+                if (!in) bl.push_back((int)i);
+            }
+            QX_CHECK((long)bl.size() == g.Vh - g.n_int, QUDAX_ERR_STATE, "boundary list size");
+            c->blist = static_cast<int *>(dalloc(c, sizeof(int) * std::max<size_t>(bl.size(), 1)));
+            QX_CUDA(cudaMemcpy(c->blist, bl.data(), sizeof(int) * bl.size(), cudaMemcpyHostToDevice));
         }
     });
     if (st != QUDAX_OK) {
@@ -976,8 +1172,7 @@ long long qudax_launch_count(const qudax_ctx *c) { return c ? c->launches : -1; 
 
 qudax_status qudax_get_partition(const qudax_ctx *c, qudax_partition *out) {
     if (!c || !out) return QUDAX_ERR_ARG;
-    const int gd[4] = {c->g.X, c->g.Y, c->g.Z, c->g.T};
-    return fill_partition(gd, c->g.nranks, c->g.rank, out);
+    return fill_partition(c->g.G, c->g.P, c->g.nranks, c->g.rank, c->g.split, c->comm, c->p2p.on, out);
 }
 
 qudax_status qudax_kernel_timing(qudax_ctx *c, int enable) {

@@ -68,7 +68,7 @@ struct qudax_ctx {
     struct GaugeCopy {
         int prec = 0, recon = 0;
         void *d[4][2] = {};
-        void *ghost[2] = {};
+        void *ghost[4][2] = {};  // backward ghost links U_mu(x - mu) at x_mu = -1 per split mu, per parity
     };
     GaugeCopy gcopy[2];
     int ncopies = 0;
@@ -82,7 +82,12 @@ struct qudax_ctx {
         size_t bytes = 0;
         void *sb = nullptr, *sf = nullptr, *gb = nullptr, *gf = nullptr;
         void *h_sb = nullptr, *h_sf = nullptr, *h_gb = nullptr, *h_gf = nullptr;
+        // partitioned X / Y / Z: projected faces per dimension (send/ghost, back/fwd)
+        size_t sbytes[3] = {};
+        void *ssb[3] = {}, *ssf[3] = {}, *sgb[3] = {}, *sgf[3] = {};
+        void *h_ssb[3] = {}, *h_ssf[3] = {}, *h_sgb[3] = {}, *h_sgf[3] = {};
     } halo[3];
+    int *blist = nullptr;  // boundary sites (complement of the interior box) when X/Y/Z is split
 
     // kernel-initiated halo over peer memory (QUDAX_HALO_P2P).  One cudaMalloc region per rank,
     // identical layout on every rank: per precision ghost_back[2], ghost_fwd[2] (sequence

@@ -84,10 +84,11 @@ __device__ __forceinline__ void unpack_spinor(const R *v, Cx<R> p[4][3]) {
 }
 
 // spatial hop: project psi with (1 + sigma gamma_mu), multiply by U (or U^dag), accumulate
-// (the projector formulas of the header, written with add_i(p, q) = p + S i q)
-template <int MU, int SIGMA, bool ADJ, typename R>
-__device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3][3], Cx<R> acc[4][3]) {
-    Cx<R> h0[3], h1[3];
+// (the projector formulas of the header, written with add_i(p, q) = p + S i q).  Split into the
+// projection and the multiply-expand so a partitioned dimension's face pack projects with
+// exactly this code and the receiving kernel finishes the hop with exactly this code.
+template <int MU, int SIGMA, typename R>
+__device__ __forceinline__ void spatial_project(const Cx<R> p[4][3], Cx<R> h0[3], Cx<R> h1[3]) {
 #pragma unroll
     for (int c = 0; c < 3; ++c) {
         if constexpr (MU == 0) {  // h0 = p0 - s i p3, h1 = p1 - s i p2
@@ -101,6 +102,10 @@ __device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3
             h1[c] = add_i<SIGMA>(p[1][c], p[3][c]);
         }
     }
+}
+template <int MU, int SIGMA, bool ADJ, typename R>
+__device__ __forceinline__ void spatial_mult_expand(const Cx<R> h0[3], const Cx<R> h1[3], const Cx<R> u[3][3],
+                                                    Cx<R> acc[4][3]) {
     Cx<R> g0[3], g1[3];
     if constexpr (ADJ) {
         su3_dag_mul(u, h0, g0);
@@ -124,6 +129,88 @@ __device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3
             acc[3][c] = add_i<-SIGMA>(acc[3][c], g1[c]);
         }
     }
+}
+template <int MU, int SIGMA, bool ADJ, typename R>
+__device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3][3], Cx<R> acc[4][3]) {
+    Cx<R> h0[3], h1[3];
+    spatial_project<MU, SIGMA>(p, h0, h1);
+    spatial_mult_expand<MU, SIGMA, ADJ>(h0, h1, u, acc);
+}
+
+// Faces of a partitioned X / Y / Z: the projected half spinor (h0, h1), 12 reals in the
+// arithmetic precision R, site-major blocks of 16-byte vectors (fs = padded face sites)
+template <typename R>
+struct SFace {
+    static constexpr int NB = (sizeof(R) == 8) ? 6 : 3;
+    static __device__ __forceinline__ void load(const void *base, long fs, long f, Cx<R> h0[3], Cx<R> h1[3]) {
+        R v[12];
+        if constexpr (sizeof(R) == 8) {
+            const double2 *p = reinterpret_cast<const double2 *>(base);
+#pragma unroll
+            for (int k = 0; k < 6; ++k) {
+                const double2 d = __ldg(p + k * fs + f);
+                v[2 * k] = d.x;
+                v[2 * k + 1] = d.y;
+            }
+        } else {
+            const float4 *p = reinterpret_cast<const float4 *>(base);
+#pragma unroll
+            for (int k = 0; k < 3; ++k) {
+                const float4 d = __ldg(p + k * fs + f);
+                v[4 * k] = d.x; v[4 * k + 1] = d.y; v[4 * k + 2] = d.z; v[4 * k + 3] = d.w;
+            }
+        }
+#pragma unroll
+        for (int c = 0; c < 3; ++c) {
+            h0[c] = cx(v[2 * c], v[2 * c + 1]);
+            h1[c] = cx(v[6 + 2 * c], v[6 + 2 * c + 1]);
+        }
+    }
+    static __device__ __forceinline__ void store(void *base, long fs, long f, const Cx<R> h0[3], const Cx<R> h1[3]) {
+        R v[12];
+#pragma unroll
+        for (int c = 0; c < 3; ++c) {
+            v[2 * c] = h0[c].r; v[2 * c + 1] = h0[c].i;
+            v[6 + 2 * c] = h1[c].r; v[6 + 2 * c + 1] = h1[c].i;
+        }
+        if constexpr (sizeof(R) == 8) {
+            double2 *p = reinterpret_cast<double2 *>(base);
+#pragma unroll
+            for (int k = 0; k < 6; ++k) p[k * fs + f] = make_double2(v[2 * k], v[2 * k + 1]);
+        } else {
+            float4 *p = reinterpret_cast<float4 *>(base);
+#pragma unroll
+            for (int k = 0; k < 3; ++k) p[k * fs + f] = make_float4(v[4 * k], v[4 * k + 1], v[4 * k + 2], v[4 * k + 3]);
+        }
+    }
+};
+// A partitioned X / Y / Z face as the receiving Dslash reads it.  fp64 / fp32: the sender's
+// spin projection (SFace).  Half: the sender's raw 16-bit record (same layout as a half spinor
+// field with stride fs, norm included; 52 B per site, less than a projected fp32 face) projected
+// here from exactly the values the unpartitioned kernel decodes.
+template <int P, int MU, int SIGMA>
+__device__ __forceinline__ void ghost_half(const void *base, long fs, long f, Cx<typename Prec<P>::R> h0[3],
+                                           Cx<typename Prec<P>::R> h1[3]) {
+    using R = typename Prec<P>::R;
+    if constexpr (P == 2) {
+        RawVec<2, 24> sv;
+        sv.template load_spinor<0>(base, fs, f);
+        R v[24];
+        Cx<R> ps[4][3];
+        sv.decode(v);
+        unpack_spinor(v, ps);
+        spatial_project<MU, SIGMA>(ps, h0, h1);
+    } else {
+        SFace<R>::load(base, fs, f, h0, h1);
+    }
+}
+// index of a site in the face of dimension mu (lexicographic over the other three local
+// coordinates, halved: the sites of one parity on a face pair up along the fastest of them)
+template <int MU>
+__device__ __forceinline__ int face_index(int x, int y, int z, int t, int X, int Y, int Z) {
+    if constexpr (MU == 0) return ((t * Z + z) * Y + y) >> 1;
+    else if constexpr (MU == 1) return ((t * Z + z) * X + x) >> 1;
+    else return ((t * Y + y) * X + x) >> 1;
 }
 
 // temporal hop: h = the 12 selected reals (upper half if UPPER); result 2 U h into the same half
@@ -281,28 +368,40 @@ template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) 
 // one output site; red[] receives this site's contribution to the optional fused reduction
 // INMODE: load mode of the neighbour spinors (0 read-only path; 2 L2-coherent, for inputs
 // written by other CTAs earlier in the same launch — the fused Mhat kernel)
-template <int P, int RECON, bool DAG, int KIND, int INMODE = 0>
+// SS: the variant for contexts with a partitioned X, Y or Z (ghost-aware spatial hops); kept a
+// separate instantiation so the unpartitioned kernels keep their register allocation
+template <int P, int RECON, bool DAG, int KIND, int INMODE = 0, bool SS = false>
 __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin, void *fout, const void *fx, int tid,
                                             double red[3], long goff = 0) {
     using R = typename Prec<P>::R;
     if (a.reverse) tid = a.nthreads - 1 - tid;
-    int i;
-    if (a.range == RANGE_ALL) i = tid;
-    else if (a.range == RANGE_INTERIOR) i = a.F + tid;
-    else if (a.range == RANGE_TAIL) {
-        const int ni = (a.T_loc - 2) * a.F;
-        const int j = tid - ni;
-        i = (tid < ni) ? a.F + tid : ((j < a.F) ? j : (a.T_loc - 1) * a.F + (j - a.F));
-    }
-    else i = (tid < a.F) ? tid : (a.T_loc - 1) * a.F + (tid - a.F);
-
     const int X = a.X, Y = a.Y, Z = a.Z, Xh = a.Xh;
-    int xh = i % Xh;
-    int r = i / Xh;
-    const int y = r % Y;
-    r /= Y;
-    const int z = r % Z;
-    const int t = r / Z;
+    int i, xh, y, z, t;
+    if (SS && a.range == RANGE_INTERIOR) {  // the interior box of a multi-dimensional split
+        int r = tid;
+        xh = r % a.bn[0] + a.blo[0];
+        r /= a.bn[0];
+        y = r % a.bn[1] + a.blo[1];
+        r /= a.bn[1];
+        z = r % a.bn[2] + a.blo[2];
+        t = r / a.bn[2] + a.blo[3];
+        i = ((t * Z + z) * Y + y) * Xh + xh;
+    } else {
+        if (a.range == RANGE_ALL) i = tid;
+        else if (a.range == RANGE_INTERIOR) i = a.F + tid;  // T-only split: t in [1, T_loc-2]
+        else if (a.range == RANGE_TAIL) {
+            const int ni = (a.T_loc - 2) * a.F;
+            const int j = tid - ni;
+            i = (tid < ni) ? a.F + tid : ((j < a.F) ? j : (a.T_loc - 1) * a.F + (j - a.F));
+        } else if (SS) i = __ldg(a.blist + tid);  // complement of the interior box
+        else i = (tid < a.F) ? tid : (a.T_loc - 1) * a.F + (tid - a.F);
+        xh = i % Xh;
+        int r = i / Xh;
+        y = r % Y;
+        r /= Y;
+        z = r % Z;
+        t = r / Z;
+    }
     const int x = 2 * xh + ((a.parity + y + z + t) & 1);
     const int p = a.parity, op = 1 - p;
     const int XY = X * Y;
@@ -339,8 +438,52 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // of the backward hop are issued before the forward hop is computed: twice the bytes in
     // flight per thread (dslash_pair).
     constexpr bool PAIR = dslash_pair<P, RECON>();
-    auto spatial = [&](auto mu_c, int nf, int nb) {
+    auto spatial = [&](auto mu_c, int coord, int Lmu, int nf, int nb) {
         constexpr int MU = decltype(mu_c)::value;
+        if (SS && ((a.smask >> MU) & 1)) {
+            // partitioned dimension: a hop off the local box reads the neighbour's projected face
+            const bool gf = (coord == Lmu - 1), gb = (coord == 0);
+            if (gf || gb) {
+                const int f = face_index<MU>(x, y, z, t, X, Y, Z);
+                Cx<R> h0[3], h1[3], u[3][3];
+                if (gf) {
+                    ghost_half<P, MU, SF>(a.sghost_fwd[MU], a.sfs[MU], f, h0, h1);
+                } else {
+                    RawVec<P, 24> sv;
+                    sv.template load_spinor<INMODE>(fin, a.stride, nf);
+                    R v[24];
+                    Cx<R> ps[4][3];
+                    sv.decode(v);
+                    unpack_spinor(v, ps);
+                    spatial_project<MU, SF>(ps, h0, h1);
+                }
+                {
+                    RawLink<P, RECON> l;
+                    l.load(a.gauge[MU][p], a.stride, i);
+                    l.decode(u);
+                }
+                spatial_mult_expand<MU, SF, false>(h0, h1, u, acc);
+                if (gb) {
+                    ghost_half<P, MU, SB>(a.sghost_back[MU], a.sfs[MU], f, h0, h1);
+                    RawLink<P, RECON> l;
+                    l.load(a.gauge_sghost[MU], a.sfs[MU], f);
+                    l.decode(u);
+                } else {
+                    RawVec<P, 24> sv;
+                    sv.template load_spinor<INMODE>(fin, a.stride, nb);
+                    R v[24];
+                    Cx<R> ps[4][3];
+                    sv.decode(v);
+                    unpack_spinor(v, ps);
+                    spatial_project<MU, SB>(ps, h0, h1);
+                    RawLink<P, RECON> l;
+                    l.load(a.gauge[MU][op], a.stride, nb);
+                    l.decode(u);
+                }
+                spatial_mult_expand<MU, SB, true>(h0, h1, u, acc);
+                return;
+            }
+        }
         RawVec<P, 24> sf, sb;
         RawLink<P, RECON> lf, lb;
         sf.template load_spinor<INMODE>(fin, a.stride, nf);
@@ -370,11 +513,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             spatial_hop<MU, SB, true>(ps, u, acc);
         }
     };
-    spatial(std::integral_constant<int, 0>{}, (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1,
+    spatial(std::integral_constant<int, 0>{}, x, X, (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1,
             (x == 0 ? lex + (X - 1) : lex - 1) >> 1);
-    spatial(std::integral_constant<int, 1>{}, (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1,
+    spatial(std::integral_constant<int, 1>{}, y, Y, (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1,
             (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1);
-    spatial(std::integral_constant<int, 2>{}, (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1,
+    spatial(std::integral_constant<int, 2>{}, z, Z, (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1,
             (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1);
 
     // ---- t direction: diagonal projectors, 12 reals per neighbour (eq. (6))
@@ -512,7 +655,7 @@ __device__ __forceinline__ long p2p_wait(const DslashArgs &a) {
     return (s_seq & 1u) ? a.p2p_pdist : 0L;
 }
 
-template <int P, int RECON, bool DAG, int KIND>
+template <int P, int RECON, bool DAG, int KIND, bool SS>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
     // one thread per output site (a one-wave grid-stride variant measured 8-25% slower: the
     // hardware CTA scheduler balances the memory-latency-bound CTAs better than a fixed wave)
@@ -531,7 +674,7 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     long goff = 0;
     // RANGE_TAIL: only CTAs holding boundary sites (the grid's last ones) wait for the halo
     if (a.p2p_flags && (a.range != RANGE_TAIL || (blk + 1) * (int)blockDim.x > (a.T_loc - 2) * a.F)) goff = p2p_wait(a);
-    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND>(a, fin, fout, fx, tid, red, goff);
+    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND, 0, SS>(a, fin, fout, fx, tid, red, goff);
     if (a.p2p_flags) {  // the last CTA to finish advances the consumed-halo counter
         __syncthreads();
         if (threadIdx.x == 0 && atomicAdd(a.p2p_ccount, 1u) == gridDim.x - 1) {
@@ -560,13 +703,13 @@ int dslash_blocks_prec(int recon, int dagger, int kind, int nthreads) {
     throw Error(QUDAX_ERR_ARG, "dslash: unsupported recon/kind");
 }
 
-template <int P>
+template <int P, bool SS = false>
 void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
     const int threads = QX_DSLASH_THREADS;
     if (a.nthreads <= 0) return;
 #define QX_DS(RC, DG, KD)                                                                       \
     if (recon == RC && dagger == DG && kind == KD) {                                            \
-        dslash_kernel<P, RC, DG, KD><<<dslash_blocks<P, RC, DG, KD>(a.nthreads) * (a.nrhs > 1 ? a.nrhs : 1), \
+        dslash_kernel<P, RC, DG, KD, SS><<<dslash_blocks<P, RC, DG, KD>(a.nthreads) * (a.nrhs > 1 ? a.nrhs : 1), \
                                        threads, 0, s>>>(a);                                     \
         return;                                                                                 \
     }

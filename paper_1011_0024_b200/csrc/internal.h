@@ -60,12 +60,24 @@ inline size_t clover_bytes(int prec, long stride) {
 
 // ----------------------------------------------------------------------------- geometry
 struct Geom {
-    int X, Y, Z, T;        // global
+    int X, Y, Z, T;        // LOCAL extents X_loc, Y_loc, Z_loc and the global T
     int T_loc, t0, rank, nranks;
     int Xh;                // X/2
-    long Vs, V, Vh, F;     // X*Y*Z, local volume, V/2, face sites = Vs/2
+    long Vs, V, Vh, F;     // X*Y*Z, local volume, V/2, T-face sites = Vs/2
     long stride, fstride;  // padded Vh, padded F
+    // process grid: rank = ((ct*Pz + cz)*Py + cy)*Px + cx
+    int G[4];              // global dims
+    int L[4];              // local dims (X, Y, Z, T_loc)
+    int P[4], c[4], o[4];  // grid, coordinates, origin
+    int nbf[4], nbb[4];    // neighbour ranks per dimension
+    int split;             // bit mu: dimension mu has ghost zones
+    long Fd[4], fsd[4];    // per-parity face sites along mu (V / L_mu / 2) and padded
+    // interior box in (xh, y, z, t) coordinates (sites whose hops never touch a ghost) and its size
+    int blo[4], bn[4];
+    long n_int;            // interior sites; Vh - n_int boundary sites
 };
+// bit mu of the dimensions whose ghosts are NOT the T face (X, Y, Z)
+inline int spatial_split(const Geom &g) { return g.split & 7; }
 
 // ----------------------------------------------------------------------------- reductions
 // device-resident BiCGstab scalars (Algorithm R), advanced by apply_coef after each reduction
@@ -98,6 +110,17 @@ struct DslashArgs {
     int X, Y, Z, T_loc, Xh;
     int Vh, F;
     long stride, fstride;
+    // partitioned X / Y / Z: bit mu of smask set -> hops off the local box
+    // in mu read spin-projected half spinors (arithmetic precision) from sghost_{back,fwd}[mu]
+    // (face layout, sfs[mu] padded sites) and the backward link from gauge_sghost[mu]
+    int smask;
+    long sfs[3];
+    const void *sghost_back[3], *sghost_fwd[3];
+    const void *gauge_sghost[3];
+    // RANGE_INTERIOR: the interior box (xh, y, z, t) = blo + [0, bn); RANGE_BOUNDARY with
+    // blist != nullptr: sites blist[0 .. nthreads) (the complement of the box)
+    int blo[4], bn[4];
+    const int *blist;
     int parity;            // output parity p
     int range;             // SiteRange
     int ghosted;           // 1: t-hops off the slab read ghost buffers; 0: periodic wrap
@@ -158,6 +181,13 @@ int dslash_blocks_f64(int recon, int dagger, int kind, int nthreads);
 int dslash_blocks_f32(int recon, int dagger, int kind, int nthreads);
 int dslash_blocks_f16(int recon, int dagger, int kind, int nthreads);
 
+// face pack of the partitioned X / Y / Z dimensions (bit mu of g.split, mu < 3): for each, the
+// x_mu = 0 face projected with the receiver's forward-hop projector -> sb[mu], the x_mu = L-1
+// face with its backward-hop projector -> sf[mu]; 12 reals per site in the arithmetic precision
+void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, const void *in, void *const sb[3],
+                         void *const sf[3], cudaStream_t s);
+// bytes of one spatial face buffer along mu
+size_t sface_bytes(int prec, long fs);
 // face pack: t_loc = 0 slice half (lower if !dagger) -> send_back; t_loc = T_loc-1 half
 // (upper if !dagger) -> send_fwd.  `in` is the Dslash input field (parity 1-p).
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back,
@@ -175,11 +205,20 @@ void launch_spinor_import(int prec, const Geom &g, int parity, const double *src
 void launch_spinor_export(int prec, const Geom &g, int parity, const void *src, double *dst, cudaStream_t s);
 void launch_spinor_convert(int dst_prec, int src_prec, const Geom &g, void *dst, const void *src, cudaStream_t s);
 
-// gauge: extended fp64 AoS [T_loc+2][4][Z][Y][X][3][3] complex (slot 0 = global t0-1,
-// slot T_loc+1 = t0+T_loc) -> per-mu, per-parity SoA (prec, recon) plus the ghost U_t(t0-1)
-// per site parity (face layout).  *bad counts links with |u01|^2+|u02|^2 < 1e-6 (recon 8).
+// gauge: extended fp64 site-major AoS ext[Et][Ez][Ey][Ex][4][3][3] complex, E_mu = L_mu + 2 for
+// split dimensions (ext index 0 = local -1, L_mu + 1 = local L_mu), L_mu otherwise.
+inline long ext_extent(const Geom &g, int mu) { return g.L[mu] + ((g.split >> mu & 1) ? 2 : 0); }
+inline long ext_sites(const Geom &g) { return ext_extent(g, 0) * ext_extent(g, 1) * ext_extent(g, 2) * ext_extent(g, 3); }
+// host-order box [4][T_loc][Z][Y][X][18] (device) -> ext interior
+void launch_ext_fill(const Geom &g, const double *box, double *ext, cudaStream_t s);
+// ext cross-section at ext index e along mu (all ext extents of the other dims) <-> buf
+void launch_ext_slice(const Geom &g, double *ext, int mu, int e, double *buf, bool to_buf, cudaStream_t s);
+long ext_slice_doubles(const Geom &g, int mu);
+// ext -> per-mu, per-parity SoA (prec, recon) plus the backward ghost links U_mu(x - mu) at
+// x_mu = 0 of every split dimension, per site parity, in face layout (ghost[mu][parity]).
+// *bad counts links with |u01|^2+|u02|^2 < 1e-6 (recon 8).
 void launch_gauge_pack2(int prec, int recon, const Geom &g, const double *ext, void *const dst[4][2],
-                        void *const ghost[2], int *bad, cudaStream_t s);
+                        void *const ghost[4][2], int *bad, cudaStream_t s);
 // clover: from the extended fp64 gauge, T = 1 + 2 kappa A and T^{-1} as two 6x6 Hermitian
 // chiral blocks per site (fp64 [Vh][72], halved for the NR rotation), both parities.
 void launch_clover_build(const Geom &g, const double *ext, double kappa, double csw, double *T[2],

@@ -115,9 +115,88 @@ void launch_spinor_convert(int pd, int ps, const Geom &g, void *dst, const void 
 }
 
 // ============================================================================ gauge
-// ext: fp64 complex [T_loc + 2][4][Z][Y][X][3][3]; slot 0 = global t0-1, slot T_loc+1 = t0+T_loc.
-__device__ __forceinline__ const double *ext_link(const double *ext, long Vs, int t_ext, int mu, long slex) {
-    return ext + (((size_t)t_ext * 4 + mu) * Vs + slex) * 18;
+// ext: fp64 site-major AoS [Et][Ez][Ey][Ex][4][3][3] complex; E_mu = L_mu + 2 on split
+// dimensions (ext index 0 = local -1, L_mu + 1 = local L_mu), else L_mu (periodic wrap in-kernel).
+struct ExtGeom {
+    int L[4], E[4], s[4];  // local extents, ext extents, 1 if split
+};
+static ExtGeom ext_geom(const Geom &g) {
+    ExtGeom e;
+    for (int m = 0; m < 4; ++m) {
+        e.L[m] = g.L[m];
+        e.s[m] = (g.split >> m) & 1;
+        e.E[m] = g.L[m] + 2 * e.s[m];
+    }
+    return e;
+}
+// link U_mu at local coordinates c (each in [-1, L] on split dims, any integer elsewhere: wrapped)
+__device__ __forceinline__ const double *ext_link(const double *ext, const ExtGeom &e, const int c[4], int mu) {
+    long idx = 0;
+    for (int d = 3; d >= 0; --d) {
+        const int v = e.s[d] ? c[d] + 1 : ((c[d] % e.L[d]) + e.L[d]) % e.L[d];
+        idx = idx * e.E[d] + v;
+    }
+    return ext + (idx * 4 + mu) * 18;
+}
+
+// host-order box [4][T][Z][Y][X][18] -> ext interior; one thread per (mu, site)
+__global__ void k_ext_fill(ExtGeom e, const double *__restrict__ box, double *__restrict__ ext) {
+    const long V = (long)e.L[0] * e.L[1] * e.L[2] * e.L[3];
+    const long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    if (k >= 4 * V) return;
+    const int mu = (int)(k / V);
+    long lex = k % V;
+    int c[4];
+    for (int d = 0; d < 4; ++d) {
+        c[d] = (int)(lex % e.L[d]);
+        lex /= e.L[d];
+    }
+    const double *src = box + k * 18;
+    double *dst = const_cast<double *>(ext_link(ext, e, c, mu));
+#pragma unroll
+    for (int j = 0; j < 18; ++j) dst[j] = src[j];
+}
+
+void launch_ext_fill(const Geom &g, const double *box, double *ext, cudaStream_t s) {
+    const int T = 128;
+    k_ext_fill<<<(int)((4 * g.V + T - 1) / T), T, 0, s>>>(ext_geom(g), box, ext);
+    QX_CUDA(cudaGetLastError());
+}
+
+long ext_slice_doubles(const Geom &g, int mu) { return ext_sites(g) / ext_extent(g, mu) * 72; }
+
+// the ext cross-section at ext index idx along mu (every ext index of the other dimensions,
+// so the halos received along earlier dimensions travel on: corners) <-> contiguous buffer
+__global__ void k_ext_slice(ExtGeom e, double *ext, int mu, int idx, double *buf, int to_buf) {
+    long n = 72;
+    for (int d = 0; d < 4; ++d)
+        if (d != mu) n *= e.E[d];
+    const long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    if (k >= n) return;
+    const int j = (int)(k % 72);
+    long r = k / 72;
+    long site = 0, mul = 1;
+    for (int d = 0; d < 4; ++d) {
+        long v;
+        if (d == mu) {
+            v = idx;
+        } else {
+            v = r % e.E[d];
+            r /= e.E[d];
+        }
+        site += v * mul;
+        mul *= e.E[d];
+    }
+    double *p = ext + site * 72 + j;
+    if (to_buf) buf[k] = *p;
+    else *p = buf[k];
+}
+
+void launch_ext_slice(const Geom &g, double *ext, int mu, int e, double *buf, bool to_buf, cudaStream_t s) {
+    const long n = ext_slice_doubles(g, mu);
+    const int T = 256;
+    k_ext_slice<<<(int)((n + T - 1) / T), T, 0, s>>>(ext_geom(g), ext, mu, e, buf, to_buf ? 1 : 0);
+    QX_CUDA(cudaGetLastError());
 }
 
 template <int P, int RECON>
@@ -173,56 +252,75 @@ __device__ void encode_store_link(const double *l /*18*/, void *base, long strid
 
 struct GaugeDst {
     void *d[4][2];
-    void *ghost[2];
+    void *ghost[4][2];
+    long Fd[4], fsd[4];
 };
 
+// coordinates of face site f (parity q) of dimension mu at x_mu = xm: the inverse of
+// dslash.cuh face_index (lexicographic over the other three coordinates, halved)
+__device__ __forceinline__ void face_site(int mu, long f, int xm, int q, const int L[4], int c[4]) {
+    c[mu] = xm;
+    const int a = (mu == 0) ? 1 : 0;             // the fastest of the other dimensions (paired)
+    const int b = (mu <= 1) ? 2 : 1, d = (mu <= 2) ? 3 : 2;
+    const int ah = L[a] / 2;
+    int ch = (int)(f % ah);
+    long r = f / ah;
+    c[b] = (int)(r % L[b]);
+    c[d] = (int)(r / L[b]);
+    c[a] = 2 * ch + ((q + xm + c[b] + c[d]) & 1);
+}
+
 template <int P, int RECON>
-__global__ void k_gauge_pack(int X, int Y, int Z, int T_loc, long Vh, long F, long stride, long fstride,
-                             const double *__restrict__ ext, GaugeDst dst, int *bad) {
-    const long Vs = (long)X * Y * Z;
+__global__ void k_gauge_pack(ExtGeom e, long Vh, long stride, const double *__restrict__ ext, GaugeDst dst, int *bad) {
     const long n_bulk = 8 * Vh;  // (mu, parity, i)
-    const long n_ghost = 2 * F;  // (parity, f)
     long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
     if (k < n_bulk) {
         const int mu = (int)(k / (2 * Vh));
         const int p = (int)((k / Vh) % 2);
         const int i = (int)(k % Vh);
-        Coord c = cb_coord(i, p, X, Y, Z);
-        const long slex = c.lex - (long)c.t * Vs;
-        encode_store_link<P, RECON>(ext_link(ext, Vs, c.t + 1, mu, slex), dst.d[mu][p], stride, i, bad);
+        Coord c = cb_coord(i, p, e.L[0], e.L[1], e.L[2]);
+        const int cc[4] = {c.x, c.y, c.z, c.t};
+        encode_store_link<P, RECON>(ext_link(ext, e, cc, mu), dst.d[mu][p], stride, i, bad);
         return;
     }
     k -= n_bulk;
-    if (k < n_ghost) {
-        // U_t at global t0 - 1 (ext slot 0), site parity q; face index f = spatial lex / 2
-        const int q = (int)(k / F);
-        const int f = (int)(k % F);
-        const int Xh = X / 2;
-        int xh = f % Xh;
-        int r = f / Xh;
-        const int y = r % Y;
-        const int z = r / Y;
-        const int x = 2 * xh + ((q + y + z + 1) & 1);  // local t = -1 is odd
-        const long slex = ((long)z * Y + y) * X + x;
-        encode_store_link<P, RECON>(ext_link(ext, Vs, 0, 3, slex), dst.ghost[q], fstride, f, bad);
+    // backward ghost links U_mu(x - mu) at local x_mu = -1 of every split dimension, per site
+    // parity q, face layout
+    for (int mu = 0; mu < 4; ++mu) {
+        if (!e.s[mu]) continue;
+        if (k < 2 * dst.Fd[mu]) {
+            const int q = (int)(k / dst.Fd[mu]);
+            const long f = k % dst.Fd[mu];
+            int c[4];
+            face_site(mu, f, -1, q, e.L, c);
+            encode_store_link<P, RECON>(ext_link(ext, e, c, mu), dst.ghost[mu][q], dst.fsd[mu], f, bad);
+            return;
+        }
+        k -= 2 * dst.Fd[mu];
     }
 }
 
 void launch_gauge_pack2(int prec, int recon, const Geom &g, const double *ext, void *const dst[4][2],
-                        void *const ghost[2], int *bad, cudaStream_t s) {
+                        void *const ghost[4][2], int *bad, cudaStream_t s) {
     GaugeDst d;
-    for (int m = 0; m < 4; ++m)
-        for (int p = 0; p < 2; ++p) d.d[m][p] = dst[m][p];
-    d.ghost[0] = ghost[0];
-    d.ghost[1] = ghost[1];
-    const long n = 8 * g.Vh + 2 * g.F;
+    long n = 8 * g.Vh;
+    for (int m = 0; m < 4; ++m) {
+        for (int p = 0; p < 2; ++p) {
+            d.d[m][p] = dst[m][p];
+            d.ghost[m][p] = ghost[m][p];
+        }
+        d.Fd[m] = g.Fd[m];
+        d.fsd[m] = g.fsd[m];
+        if (g.split >> m & 1) n += 2 * g.Fd[m];
+    }
     const int T = 128;
     const int b = nblk(n, T);
-#define QX_GP(PP, RR)                                                                                          \
-    if (prec == PP && recon == RR) {                                                                           \
-        k_gauge_pack<PP, RR><<<b, T, 0, s>>>(g.X, g.Y, g.Z, g.T_loc, g.Vh, g.F, g.stride, g.fstride, ext, d, bad); \
-        QX_CUDA(cudaGetLastError());                                                                           \
-        return;                                                                                                \
+    const ExtGeom e = ext_geom(g);
+#define QX_GP(PP, RR)                                                               \
+    if (prec == PP && recon == RR) {                                                \
+        k_gauge_pack<PP, RR><<<b, T, 0, s>>>(e, g.Vh, g.stride, ext, d, bad);       \
+        QX_CUDA(cudaGetLastError());                                                \
+        return;                                                                     \
     }
     QX_GP(8, 18) QX_GP(8, 12) QX_GP(8, 8) QX_GP(4, 18) QX_GP(4, 12) QX_GP(4, 8) QX_GP(2, 18) QX_GP(2, 12) QX_GP(2, 8)
 #undef QX_GP
@@ -302,28 +400,26 @@ __device__ void store_herm6_half(const Cd m[6][6], double *out) {
 }
 
 // one thread per local site (both parities); T[p], Tinv[p]: fp64 [Vh][72]
-__global__ void k_clover_build(int X, int Y, int Z, int T_loc, double kappa, double csw, const double *__restrict__ ext,
+__global__ void k_clover_build(ExtGeom e, double kappa, double csw, const double *__restrict__ ext,
                                double *T0, double *T1, double *I0, double *I1, int *bad) {
-    const long Vs = (long)X * Y * Z;
-    const long V = Vs * T_loc;
+    const int X = e.L[0], Y = e.L[1];
+    const long Vs = (long)X * Y * e.L[2];
+    const long V = Vs * e.L[3];
     const long lexl = (long)blockIdx.x * blockDim.x + threadIdx.x;
     if (lexl >= V) return;
     int c[4];
     c[0] = (int)(lexl % X);
     c[1] = (int)((lexl / X) % Y);
-    c[2] = (int)((lexl / ((long)X * Y)) % Z);
+    c[2] = (int)((lexl / ((long)X * Y)) % e.L[2]);
     c[3] = (int)(lexl / Vs);
-    const int dims[4] = {X, Y, Z, T_loc};
     const int parity = (c[0] + c[1] + c[2] + c[3]) & 1;
     const long cb = lexl >> 1;
-    // link U_mu at (site + shifts), t in ext coordinates (t_ext = t + 1), spatial periodic
+    // link U_mu at (site + shifts): halo of split dimensions, periodic wrap of the others
     auto L = [&](int mu, int dm, int dmv, int nu, int dn) -> M3 {
         int s[4] = {c[0], c[1], c[2], c[3]};
         s[dmv] += dm;
         s[nu] += dn;
-        for (int d = 0; d < 3; ++d) s[d] = (s[d] + dims[d]) % dims[d];
-        const long slex = ((long)s[2] * Y + s[1]) * X + s[0];
-        return load_m3(ext_link(ext, Vs, s[3] + 1, mu, slex));
+        return load_m3(ext_link(ext, e, s, mu));
     };
     // block-diagonal chiral pieces of sum_{mu<nu} gamma_mu gamma_nu (x) F_munu
     Cd Bup[6][6], Blo[6][6];
@@ -385,7 +481,7 @@ __global__ void k_clover_build(int X, int Y, int Z, int T_loc, double kappa, dou
 void launch_clover_build(const Geom &g, const double *ext, double kappa, double csw, double *T[2], double *Tinv[2],
                          int *bad, cudaStream_t s) {
     const int TB = 64;
-    k_clover_build<<<nblk(g.V, TB), TB, 0, s>>>(g.X, g.Y, g.Z, g.T_loc, kappa, csw, ext, T[0], T[1], Tinv[0], Tinv[1], bad);
+    k_clover_build<<<nblk(g.V, TB), TB, 0, s>>>(ext_geom(g), kappa, csw, ext, T[0], T[1], Tinv[0], Tinv[1], bad);
     QX_CUDA(cudaGetLastError());
 }
 
@@ -539,6 +635,97 @@ void launch_pack_faces_p2p(int prec, int dagger, const Geom &g, const void *in, 
     else QX_PP(2);
 #undef QX_PP
     QX_CUDA(cudaGetLastError());
+}
+
+// Faces of the partitioned X / Y / Z: the x_mu = 0 face goes backward and
+// feeds the receiver's FORWARD hop, so it is projected with (1 + SF gamma_mu); the x_mu = L-1
+// face goes forward and feeds the backward hop (1 + SB gamma_mu).  Projection by the Dslash's
+// own spatial_project on the values the Dslash would decode: the receiver finishes the hop
+// bit-identically to the unpartitioned kernel.  Half precision ships the raw 16-bit record and
+// its norm instead (52 B per site vs 48 B projected in fp32); the receiver projects it
+// (dslash.cuh ghost_half) — measured: a projected half face differed from the unsplit kernel
+// by one half-precision quantum on ~4% of the Y-face sites.
+struct SPackArgs {
+    int L[4];
+    int mask;       // split spatial dims
+    int q;          // parity of the packed (input) field
+    long Fd[3], fsd[3], stride;
+    void *sb[3], *sf[3];
+};
+template <int P, bool DAG>
+__global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *__restrict__ in) {
+    using R = typename Prec<P>::R;
+    long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    int mu = 0;
+    for (; mu < 3; ++mu) {
+        if (!(a.mask >> mu & 1)) continue;
+        if (k < 2 * a.Fd[mu]) break;
+        k -= 2 * a.Fd[mu];
+    }
+    if (mu == 3) return;
+    const bool fwd = k >= a.Fd[mu];
+    const long f = fwd ? k - a.Fd[mu] : k;
+    int c[4];
+    face_site(mu, f, fwd ? a.L[mu] - 1 : 0, a.q, a.L, c);
+    const long i = (((long)(c[3] * a.L[2] + c[2]) * a.L[1] + c[1]) * a.L[0] + c[0]) >> 1;
+    void *dst = fwd ? a.sf[mu] : a.sb[mu];
+    if constexpr (P == 2) {  // half: the raw record + norm (bits only; the receiver projects)
+        for (int hf = 0; hf < 2; ++hf) {
+            reinterpret_cast<uint4 *>(mptr(dst, h_spinor_u(a.fsd[mu], hf)))[f] =
+                reinterpret_cast<const uint4 *>(cptr(in, h_spinor_u(a.stride, hf)))[i];
+            reinterpret_cast<uint2 *>(mptr(dst, h_spinor_v(a.fsd[mu], hf)))[f] =
+                reinterpret_cast<const uint2 *>(cptr(in, h_spinor_v(a.stride, hf)))[i];
+        }
+        SpinorIO<2>::norms(dst, a.fsd[mu])[f] = SpinorIO<2>::norms(in, a.stride)[i];
+        return;
+    }
+    RawVec<P, 24> raw;
+    raw.template load_spinor<0>(in, a.stride, i);
+    R v[24];
+    Cx<R> ps[4][3], h0[3], h1[3];
+    raw.decode(v);
+    unpack_spinor(v, ps);
+    constexpr int SF = DAG ? +1 : -1, SB = -SF;
+    if (mu == 0) {
+        if (fwd) spatial_project<0, SB>(ps, h0, h1); else spatial_project<0, SF>(ps, h0, h1);
+    } else if (mu == 1) {
+        if (fwd) spatial_project<1, SB>(ps, h0, h1); else spatial_project<1, SF>(ps, h0, h1);
+    } else {
+        if (fwd) spatial_project<2, SB>(ps, h0, h1); else spatial_project<2, SF>(ps, h0, h1);
+    }
+    SFace<R>::store(dst, a.fsd[mu], f, h0, h1);
+}
+
+size_t sface_bytes(int prec, long fs) { return prec == 2 ? spinor_bytes(2, fs) : (size_t)12 * prec * fs; }
+
+void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, const void *in, void *const sb[3],
+                         void *const sf[3], cudaStream_t s) {
+    SPackArgs a{};
+    long n = 0;
+    for (int m = 0; m < 4; ++m) a.L[m] = g.L[m];
+    a.mask = spatial_split(g);
+    a.q = in_parity;
+    a.stride = g.stride;
+    for (int m = 0; m < 3; ++m) {
+        a.Fd[m] = g.Fd[m];
+        a.fsd[m] = g.fsd[m];
+        a.sb[m] = sb[m];
+        a.sf[m] = sf[m];
+        if (a.mask >> m & 1) n += 2 * g.Fd[m];
+    }
+    if (!n) return;
+    const int T = 128;
+    const int b = nblk(n, T);
+#define QX_PS(PP)                                                                  \
+    if (prec == PP) {                                                              \
+        if (dagger) k_pack_spatial<PP, true><<<b, T, 0, s>>>(a, in);               \
+        else k_pack_spatial<PP, false><<<b, T, 0, s>>>(a, in);                     \
+        QX_CUDA(cudaGetLastError());                                               \
+        return;                                                                    \
+    }
+    QX_PS(8) QX_PS(4) QX_PS(2)
+#undef QX_PS
+    throw Error(QUDAX_ERR_ARG, "pack spatial: bad precision");
 }
 
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back, void *send_fwd,

@@ -35,8 +35,8 @@ class QudaxError(RuntimeError):
 
 
 # ----------------------------------------------------------------------------- ctypes structs
-EXCHANGE_FN = ctypes.CFUNCTYPE(ctypes.c_int, ctypes.c_void_p, ctypes.c_void_p, ctypes.c_void_p, ctypes.c_void_p,
-                               ctypes.c_size_t, ctypes.c_void_p)
+EXCHANGE_FN = ctypes.CFUNCTYPE(ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_void_p, ctypes.c_void_p,
+                               ctypes.c_void_p, ctypes.c_void_p, ctypes.c_size_t, ctypes.c_void_p)
 ALLREDUCE_FN = ctypes.CFUNCTYPE(ctypes.c_int, ctypes.POINTER(ctypes.c_double), ctypes.c_int, ctypes.c_void_p)
 ALLOC_FN = ctypes.CFUNCTYPE(ctypes.c_void_p, ctypes.c_size_t, ctypes.c_void_p)
 FREE_FN = ctypes.CFUNCTYPE(None, ctypes.c_void_p, ctypes.c_void_p)
@@ -48,7 +48,7 @@ class InitParam(ctypes.Structure):
                 ("nccl_id", ctypes.c_void_p), ("stream", ctypes.c_size_t),
                 ("dev_alloc", ALLOC_FN), ("dev_free", FREE_FN), ("alloc_user", ctypes.c_void_p),
                 ("host_exchange", EXCHANGE_FN), ("host_allreduce", ALLREDUCE_FN), ("comm_user", ctypes.c_void_p),
-                ("halo", ctypes.c_int)]
+                ("halo", ctypes.c_int), ("proc_grid", ctypes.c_int * 4), ("split_mask", ctypes.c_int)]
 
 
 class GaugeParam(ctypes.Structure):
@@ -88,10 +88,16 @@ class Partition(ctypes.Structure):
     _fields_ = [("T_loc", ctypes.c_int), ("t0", ctypes.c_int), ("rank_fwd", ctypes.c_int),
                 ("rank_back", ctypes.c_int), ("V_loc", ctypes.c_long), ("V_h", ctypes.c_long),
                 ("V_s", ctypes.c_long), ("face_sites", ctypes.c_long), ("applies_bc_fwd", ctypes.c_int),
-                ("applies_bc_back", ctypes.c_int), ("face_bytes", ctypes.c_size_t * 3)]
+                ("applies_bc_back", ctypes.c_int), ("face_bytes", ctypes.c_size_t * 3),
+                ("proc_grid", ctypes.c_int * 4), ("coords", ctypes.c_int * 4), ("local_dims", ctypes.c_int * 4),
+                ("origin", ctypes.c_int * 4), ("nb_fwd", ctypes.c_int * 4), ("nb_back", ctypes.c_int * 4),
+                ("split_mask", ctypes.c_int), ("face_sites_dim", ctypes.c_long * 4)]
 
     def as_dict(self):
-        d = {k: getattr(self, k) for k, _ in self._fields_ if k != "face_bytes"}
+        d = {}
+        for k, _ in self._fields_:
+            v = getattr(self, k)
+            d[k] = tuple(v) if k not in ("face_bytes",) and hasattr(v, "__len__") else v
         d["face_bytes"] = {"half": self.face_bytes[0], "single": self.face_bytes[1], "double": self.face_bytes[2]}
         return d
 
@@ -104,7 +110,8 @@ _DP = ctypes.POINTER(ctypes.c_double)
 SIGNATURES = {
     "qudax_abi_version": ([], _I),
     "qudax_status_string": ([_I], ctypes.c_char_p),
-    "qudax_partition_info": ([ctypes.POINTER(ctypes.c_int), _I, _I, ctypes.POINTER(Partition)], _I),
+    "qudax_partition_info": ([ctypes.POINTER(ctypes.c_int), ctypes.POINTER(ctypes.c_int), _I, _I, _I,
+                              ctypes.POINTER(Partition)], _I),
     "qudax_model": ([_I, _I, _I, ctypes.POINTER(SiteModel)], _I),
     "qudax_nccl_unique_id": ([_P], _I),
     "qudax_init": ([ctypes.POINTER(_P), ctypes.POINTER(InitParam)], _I),
@@ -157,10 +164,12 @@ def status_string(s):
     return lib().qudax_status_string(int(s)).decode()
 
 
-def partition_info(global_dims, nranks, rank):
+def partition_info(global_dims, nranks, rank, proc_grid=None, split_mask=0):
+    """Rank bookkeeping of a process grid (default 1 x 1 x 1 x nranks: T slabs)."""
     out = Partition()
     dims = (ctypes.c_int * 4)(*global_dims)
-    st = lib().qudax_partition_info(dims, int(nranks), int(rank), ctypes.byref(out))
+    grid = (ctypes.c_int * 4)(*proc_grid) if proc_grid is not None else None
+    st = lib().qudax_partition_info(dims, grid, int(nranks), int(rank), int(split_mask), ctypes.byref(out))
     if st:
         raise QudaxError(st, "partition_info")
     return out.as_dict()
@@ -201,10 +210,8 @@ def make_gloo_transport(group=None):
         arr = np.ctypeslib.as_array((ctypes.c_uint8 * n).from_address(ptr))
         return torch.from_numpy(arr)
 
-    def exchange(send_fwd, send_back, recv_back, recv_fwd, nbytes, _user):
+    def exchange(fwd, back, send_fwd, send_back, recv_back, recv_fwd, nbytes, _user):
         try:
-            r, n = dist.get_rank(group), dist.get_world_size(group)
-            fwd, back = (r + 1) % n, (r - 1) % n
             sf, sb = as_tensor(send_fwd, nbytes), as_tensor(send_back, nbytes)
             rb, rf = as_tensor(recv_back, nbytes), as_tensor(recv_fwd, nbytes)
             ops = [dist.P2POp(dist.isend, sf, fwd, group, tag=0), dist.P2POp(dist.irecv, rb, back, group, tag=0),
@@ -237,7 +244,7 @@ class Context:
     spinor_bytes(prec) bytes holding one parity in the library's layout."""
 
     def __init__(self, global_dims, nranks=1, rank=0, device=0, comm=COMM_NONE, overlap=True, nccl_id=None,
-                 stream=None, torch_allocator=True, transport=None, halo=HALO_COMM):
+                 stream=None, torch_allocator=True, transport=None, halo=HALO_COMM, proc_grid=None, split_mask=0):
         import torch
         self._torch = torch
         self.global_dims = tuple(int(d) for d in global_dims)
@@ -250,6 +257,9 @@ class Context:
         p.global_dims = (ctypes.c_int * 4)(*self.global_dims)
         p.nranks, p.rank, p.device, p.comm, p.overlap = int(nranks), int(rank), self.device, int(comm), int(bool(overlap))
         p.halo = int(halo)
+        if proc_grid is not None:
+            p.proc_grid = (ctypes.c_int * 4)(*proc_grid)
+        p.split_mask = int(split_mask)
         self._id = None
         if comm == COMM_NCCL:
             self._id = ctypes.create_string_buffer(bytes(nccl_id), 128)
@@ -282,8 +292,7 @@ class Context:
         part = Partition()
         self._check(lib().qudax_get_partition(self._h, ctypes.byref(part)))
         self.partition = part.as_dict()
-        X, Y, Z, _ = self.global_dims
-        self.local_dims = (X, Y, Z, self.partition["T_loc"])
+        self.local_dims = tuple(self.partition["local_dims"])
 
     # -- plumbing
     def _check(self, st, ctx=True):

@@ -1,6 +1,7 @@
 """Multi-rank worker (launched by tests/gpu/test_multirank.py through torchrun).
 
-Every rank drives one qudax context on ITS slab of a T-partitioned global lattice.  All ranks
+Every rank drives one qudax context on ITS box of a global lattice split over a process grid
+(default T slabs; --grid Px,Py,Pz,Pt for the multi-dimensional split).  All ranks
 may share one GPU (the QUDAX_COMM_HOST transport stages faces through pinned host memory and
 exchanges them with torch.distributed/gloo — the paper's non-overlapped strategy),
 or use NCCL when the ranks own distinct GPUs.  Rank 0 gathers the slabs and compares them
@@ -32,26 +33,36 @@ def main():
     ap.add_argument("--dims", default="8,4,6,16")
     ap.add_argument("--same-gpu", type=int, default=1)
     ap.add_argument("--halo", default="comm", help="comm | p2p (kernel-initiated over CUDA IPC peer memory)")
+    ap.add_argument("--grid", default="", help="process grid Px,Py,Pz,Pt (default 1,1,1,N: T slabs)")
     args = ap.parse_args()
     dims = tuple(int(v) for v in args.dims.split(","))
     dist.init_process_group("gloo")
     rank, n = dist.get_rank(), dist.get_world_size()
     device = 0 if args.same_gpu else rank
     torch.cuda.set_device(device)
-    T_loc = dims[3] // n
-    t0 = rank * T_loc
-    U = qgen.gauge(dims, 1301, eps=-1.0, t_begin=t0, nt=T_loc)
-    psi = qgen.spinor(dims, 1302, t_begin=t0, nt=T_loc)
-    xin = qgen.spinor(dims, 1303, t_begin=t0, nt=T_loc)
-    result = {"rank": rank, "n": n, "comm": args.comm, "halo": args.halo, "ok": True, "checks": {}}
+    grid = tuple(int(v) for v in args.grid.split(",")) if args.grid else (1, 1, 1, n)
+    part = qudax.partition_info(dims, n, rank, proc_grid=grid)
+    L, o = part["local_dims"], part["origin"]
+
+    def box(a, lead=0):
+        """this rank's box of a global [.., T, Z, Y, X, ...] array (lead = leading axes)"""
+        sl = (slice(None),) * lead + tuple(slice(o[m], o[m] + L[m]) for m in (3, 2, 1, 0))
+        return np.ascontiguousarray(a[sl])
+    Ug_all = qgen.gauge(dims, 1301, eps=-1.0)
+    U = box(Ug_all, 1)
+    psi = box(qgen.spinor(dims, 1302))
+    xin = box(qgen.spinor(dims, 1303))
+    result = {"rank": rank, "n": n, "comm": args.comm, "halo": args.halo, "grid": grid, "ok": True, "checks": {}}
     halo = qudax.HALO_P2P if args.halo == "p2p" else qudax.HALO_COMM
     if args.comm == "nccl":
         obj = [qudax.nccl_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(obj, src=0)
         ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_NCCL, nccl_id=obj[0],
-                            halo=halo)
+                            halo=halo, proc_grid=grid)
     else:
-        ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_HOST, halo=halo)
+        ctx = qudax.Context(dims, nranks=n, rank=rank, device=device, comm=qudax.COMM_HOST, halo=halo,
+                            proc_grid=grid)
+    assert ctx.local_dims == L
     outs = {}
     for prec, recon in ((8, 18), (4, 12), (2, 12)):
         ctx.gauge_load(U, 0.12, 1.0, prec=prec, recon=recon, t_boundary=-1)
@@ -70,15 +81,25 @@ def main():
         outs[(prec, "norm2")] = ctx.norm2(fb, prec)
     # solver across ranks (global reductions through the transport)
     ctx.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12, t_boundary=-1)
-    b = qgen.point_source(dims, 0, 1, t_begin=t0, nt=T_loc)
+    b = box(qgen.point_source(dims, 0, 1))
     x, st = ctx.solve(b, tol=1e-10, delta=0.1, maxiter=2000, prec=8, prec_sloppy=4)
     outs["solve_x"] = x
     outs["solve_stats"] = st
+    outs["origin"] = o
     ctx.close()
 
     # gather slabs to rank 0
     gathered = [None] * n
     dist.gather_object(outs, gathered if rank == 0 else None, dst=0)
+    def assemble(key):
+        """global array from the ranks' boxes"""
+        first = gathered[0][key]
+        out = np.empty((dims[3], dims[2], dims[1], dims[0]) + first.shape[4:], dtype=first.dtype)
+        for g in gathered:
+            og = g["origin"]
+            out[og[3]:og[3] + L[3], og[2]:og[2] + L[2], og[1]:og[1] + L[1], og[0]:og[0] + L[0]] = g[key]
+        return out
+
     if rank == 0:
         ref = qudax.Context(dims, device=device)
         Ug = qgen.gauge(dims, 1301, eps=-1.0)
@@ -93,14 +114,14 @@ def main():
                     for kind in (0, 1, 2):
                         ref.dslash(fo, fi, prec, p, dagger=dag, kind=kind, x=fx, a=-0.3)
                         want = ref.spinor_store(fo, prec, p)
-                        got = np.concatenate([g[(prec, p, dag, kind)] for g in gathered], axis=0)
+                        got = assemble((prec, p, dag, kind))
                         same = bool(np.array_equal(got, want))
                         result["checks"][f"dslash p{prec} par{p} dag{dag} kind{kind}"] = same
                         result["ok"] &= same
             fa, fb = ref.new_field(prec), ref.new_field(prec)
             ref.spinor_load(fa, prec, 0, pg)
             ref.mdagm(fb, fa, prec)
-            got = np.concatenate([g[(prec, "mdagm")] for g in gathered], axis=0)
+            got = assemble((prec, "mdagm"))
             same = bool(np.array_equal(got, ref.spinor_store(fb, prec, 0)))
             result["checks"][f"mdagm p{prec}"] = same
             result["ok"] &= same
@@ -113,7 +134,7 @@ def main():
         # solver: oracle true residual of the gathered solution
         import oracle
         wc = oracle.WilsonClover(Ug, 0.124, 1.0, -1.0)
-        xg_ = np.concatenate([g["solve_x"] for g in gathered], axis=0)
+        xg_ = assemble("solve_x")
         bg = qgen.point_source(dims, 0, 1)
         res = float(np.linalg.norm(wc.M(xg_) - bg) / np.linalg.norm(bg))
         result["solve"] = {"oracle_true_res": res, "stats": gathered[0]["solve_stats"]}

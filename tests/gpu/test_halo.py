@@ -54,6 +54,52 @@ def test_loopback_bitwise(torch_cuda, prec, overlap, halo):
     loop.close()
 
 
+@pytest.mark.parametrize("mask", [0b0100, 0b0110, 0b0001, 0b1111])
+@pytest.mark.parametrize("prec", [8, 4, 2])
+def test_loopback_split_dims_bitwise(torch_cuda, prec, mask):
+    """Multi-dimensional split path at N=1: every dimension in `mask` sends
+    its faces to itself through NCCL (X/Y/Z faces spin-projected by the pack kernel in the
+    arithmetic precision), interior box + boundary-list kernels; bitwise = unsplit."""
+    dims = (8, 4, 6, 8)
+    U = qgen.gauge(dims, 1221)
+    psi = qgen.spinor(dims, 1222)
+    x = qgen.spinor(dims, 1223)
+    ref = qudax.Context(dims)
+    loop = qudax.Context(dims, comm=qudax.COMM_NCCL, nccl_id=qudax.nccl_unique_id(), split_mask=mask)
+    assert loop.partition["split_mask"] == mask
+    outs = {}
+    for name, c in (("ref", ref), ("loop", loop)):
+        c.gauge_load(U, 0.12, 1.0, prec=prec, recon=12)
+        fi, fo, fx = c.new_field(prec), c.new_field(prec), c.new_field(prec)
+        res = []
+        for p in (0, 1):
+            c.spinor_load(fi, prec, 1 - p, psi)
+            c.spinor_load(fx, prec, p, x)
+            for dagger in (False, True):
+                for kind in (0, 1, 2, 3):
+                    c.dslash(fo, fi, prec, p, dagger=dagger, kind=kind, x=fx, a=-0.2)
+                    c.sync()
+                    res.append(fo.cpu().numpy().copy())
+        fa, fb, fc = c.new_field(prec), c.new_field(prec), c.new_field(prec)
+        c.spinor_load(fa, prec, 0, psi)
+        c.matpc(fb, fa, prec)
+        c.matpc(fc, fb, prec, dagger=True)
+        c.mdagm(fb, fc, prec)
+        c.sync()
+        res.append(fb.cpu().numpy().copy())
+        outs[name] = res
+    for k, (a, b) in enumerate(zip(outs["ref"], outs["loop"])):
+        assert np.array_equal(a, b), k
+    ref.close()
+    loop.close()
+
+
+def test_p2p_rejects_spatial_split(torch_cuda):
+    with pytest.raises(qudax.QudaxError) as e:
+        qudax.Context((8, 4, 6, 8), halo=qudax.HALO_P2P, split_mask=0b1100)
+    assert e.value.status == 5
+
+
 def test_p2p_loopback_solve(torch_cuda):
     """Mixed-precision solve through the kernel-initiated halo (graph replay included): same
     iterations and residual history as the unsplit context (bitwise operators)."""
@@ -69,3 +115,21 @@ def test_p2p_loopback_solve(torch_cuda):
         c.close()
     assert res["ref"][1]["iters"] == res["p2p"][1]["iters"]
     assert np.array_equal(res["ref"][0], res["p2p"][0])
+
+
+def test_loopback_split_dims_solve(torch_cuda):
+    """Mixed-precision solve with Y, Z and T split in loopback (NCCL to self, CUDA-graph
+    replay of the iteration included): bitwise the unsplit solve."""
+    dims = (8, 4, 4, 16)
+    U = qgen.gauge(dims, 1231, eps=0.1)
+    b = qgen.point_source(dims, 1, 2)
+    res = {}
+    for name, kw in (("ref", {}), ("split", {"comm": qudax.COMM_NCCL, "nccl_id": qudax.nccl_unique_id(),
+                                               "split_mask": 0b1110})):
+        c = qudax.Context(dims, **kw)
+        c.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+        x, st = c.solve(b, tol=1e-12, delta=0.1, maxiter=1000, prec=8, prec_sloppy=4)
+        res[name] = (x, st)
+        c.close()
+    assert res["ref"][1]["iters"] == res["split"][1]["iters"]
+    assert np.array_equal(res["ref"][0], res["split"][0])

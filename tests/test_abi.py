@@ -28,7 +28,7 @@ def test_library_exports_every_header_symbol():
 
 
 def test_abi_version_and_status_strings():
-    assert qudax.lib().qudax_abi_version() == 2
+    assert qudax.lib().qudax_abi_version() == 3
     assert qudax.status_string(0) == "ok"
     assert "unsupported" in qudax.status_string(5)
 
@@ -67,6 +67,42 @@ def test_partition_info():
                 ((4, 4, 4, 8), 2, 2)]:
         with pytest.raises(qudax.QudaxError):
             qudax.partition_info(*bad)
+
+
+def test_partition_grid():
+    """Process grids: rank = ((ct Pz + cz) Py + cy) Px + cx, local boxes
+    tile the global lattice, neighbours are mutual, faces are V_loc / L_mu / 2 sites."""
+    dims, grid = (8, 4, 8, 16), (2, 1, 2, 2)
+    n = 8
+    parts = [qudax.partition_info(dims, n, r, proc_grid=grid) for r in range(n)]
+    seen = set()
+    for r, p in enumerate(parts):
+        assert p["proc_grid"] == grid and p["local_dims"] == (4, 4, 4, 8)
+        cx, cy, cz, ct = p["coords"]
+        assert r == ((ct * grid[2] + cz) * grid[1] + cy) * grid[0] + cx
+        assert p["origin"] == tuple(c * l for c, l in zip(p["coords"], p["local_dims"]))
+        seen.add(p["origin"])
+        assert p["split_mask"] == 0b1101  # x, z, t split; y not
+        for mu in range(4):
+            assert parts[p["nb_fwd"][mu]]["nb_back"][mu] == r
+            q = parts[p["nb_fwd"][mu]]
+            for nu in range(4):  # the forward neighbour differs in coordinate mu only
+                want = (p["coords"][nu] + (nu == mu)) % grid[nu]
+                assert q["coords"][nu] == want
+            assert p["face_sites_dim"][mu] == 4 * 4 * 4 * 8 // p["local_dims"][mu] // 2
+        assert p["T_loc"] == 8 and p["t0"] == ct * 8
+        assert p["applies_bc_fwd"] == (ct == 1) and p["applies_bc_back"] == (ct == 0)
+    assert len(seen) == n
+    # default grid = T slabs; loopback mask on one rank; bad grids
+    assert qudax.partition_info((4, 4, 4, 8), 2, 1)["proc_grid"] == (1, 1, 1, 2)
+    assert qudax.partition_info((4, 4, 4, 8), 1, 0, split_mask=0b0100)["split_mask"] == 0b0100
+    for args, kw in [(((4, 4, 4, 8), 4, 0), {"proc_grid": (1, 1, 2, 1)}),     # product != nranks
+                     (((4, 4, 6, 8), 2, 0), {"proc_grid": (1, 1, 2, 1)}),     # Z_loc = 3 odd
+                     (((4, 4, 4, 8), 2, 0), {"proc_grid": (1, 1, 2, 1), "split_mask": 8}),  # misses z
+                     (((4, 3, 4, 8), 2, 0), {"proc_grid": (2, 1, 1, 1)}),     # X split needs Y even
+                     (((4, 4, 4, 8), 1, 0), {"split_mask": 16})]:
+        with pytest.raises(qudax.QudaxError):
+            qudax.partition_info(*args, **kw)
 
 
 def test_init_without_gpu_fails_loudly():

@@ -50,8 +50,8 @@ def _w_transport(rank, n, port, q):
     sf = np.full(nb, rank * 2 + 1, dtype=np.uint8)   # goes forward to rank+1
     sb = np.full(nb, rank * 2 + 2, dtype=np.uint8)   # goes backward to rank-1
     rb, rf = np.zeros(nb, np.uint8), np.zeros(nb, np.uint8)
-    rc = ex(sf.ctypes.data, sb.ctypes.data, rb.ctypes.data, rf.ctypes.data, nb, None)
     back, fwd = (rank - 1) % n, (rank + 1) % n
+    rc = ex(fwd, back, sf.ctypes.data, sb.ctypes.data, rb.ctypes.data, rf.ctypes.data, nb, None)
     ok = rc == 0 and np.all(rb == back * 2 + 1) and np.all(rf == fwd * 2 + 2)
     vals = np.array([rank + 1.0, 2.0 * rank], dtype=np.float64)
     rc2 = ar(vals.ctypes.data_as(ctypes.POINTER(ctypes.c_double)), 2, None)
