@@ -30,8 +30,11 @@ def main():
     ap.add_argument("--nrhs", default="", help="comma list: also time multi-RHS Mhat for these counts")
     args = ap.parse_args()
     dims = tuple(int(v) for v in args.dims.split(","))
-    peak = json.load(open(os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))),
-                                       "MEASURED_PEAKS.json")))["hbm_gbs"]
+    try:
+        peak = json.load(open(os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))),
+                                           "MEASURED_PEAKS.json")))["hbm_gbs"]
+    except OSError:  # driver-written per pod; else the profiling guide's fallback
+        peak = 6650.0
     U = qgen.gauge(dims, 1005, eps=-1.0)
     psi = qgen.spinor(dims, 2005)
     ctx = qudax.Context(dims)
