@@ -182,6 +182,13 @@ __device__ __forceinline__ float2 dq2(uint32_t w, float scale) {
                                  __uint_as_float(__byte_perm(w, kHalfMagic, 0x7632)));
     return __fmul2_rn(bc(scale), __fadd2_rn(b, bc(-kHalfBias)));
 }
+// both values of a stored word as the integers they hold (no scale): 2 PRMT + FADD2.  The
+// deferred-scale half Dslash multiplies the per-site scale into the accumulation instead.
+__device__ __forceinline__ float2 dq2_q(uint32_t w) {
+    const float2 b = make_float2(__uint_as_float(__byte_perm(w, kHalfMagic, 0x7610)),
+                                 __uint_as_float(__byte_perm(w, kHalfMagic, 0x7632)));
+    return __fadd2_rn(b, bc(-kHalfBias));
+}
 // two already-scaled floats -> packed offset-binary pair (round to nearest even)
 __device__ __forceinline__ uint32_t f32x2_to_i16x2(float a, float b) {
     const uint32_t ia = __float_as_uint(__fadd_rn(a, 12615680.0f));  // 1.5*2^23 + 2^15
@@ -234,6 +241,15 @@ struct H12 {
 #pragma unroll
         for (int k = 0; k < 6; ++k) {
             const float2 d = dq2(w[k], scale);
+            out[2 * k] = d.x;
+            out[2 * k + 1] = d.y;
+        }
+    }
+    __device__ __forceinline__ void decode_q(float *out) const {
+        const uint32_t w[6] = {u.x, u.y, u.z, u.w, v.x, v.y};
+#pragma unroll
+        for (int k = 0; k < 6; ++k) {
+            const float2 d = dq2_q(w[k]);
             out[2 * k] = d.x;
             out[2 * k + 1] = d.y;
         }
@@ -386,6 +402,28 @@ struct HLink {
         }
         if constexpr (kW) {
             const float2 a = dq2(w, kHalfInv);
+            raw[RECON - 2] = a.x;
+            raw[RECON - 1] = a.y;
+        }
+    }
+    // the stored integers (link = kHalfInv * raw)
+    __device__ __forceinline__ void decode_q(float *raw) const {
+#pragma unroll
+        for (int k = 0; k < N16; ++k) {
+            const uint32_t q[4] = {u[k].x, u[k].y, u[k].z, u[k].w};
+#pragma unroll
+            for (int j = 0; j < 4; ++j) {
+                const float2 d = dq2_q(q[j]);
+                raw[8 * k + 2 * j] = d.x;
+                raw[8 * k + 2 * j + 1] = d.y;
+            }
+        }
+        if constexpr (kV) {
+            const float2 a = dq2_q(v.x), b = dq2_q(v.y);
+            raw[8 * N16] = a.x; raw[8 * N16 + 1] = a.y; raw[8 * N16 + 2] = b.x; raw[8 * N16 + 3] = b.y;
+        }
+        if constexpr (kW) {
+            const float2 a = dq2_q(w);
             raw[RECON - 2] = a.x;
             raw[RECON - 1] = a.y;
         }
@@ -548,6 +586,12 @@ struct RawVec {
             for (int r = 0; r < NREAL / 12; ++r) h[r].decode(scale, out + 12 * r);
         }
     }
+    // half: the stored integers; value = scale() * out
+    __device__ __forceinline__ void decode_q(float *out) const {
+#pragma unroll
+        for (int r = 0; r < NREAL / 12; ++r) h[r].decode_q(out + 12 * r);
+    }
+    __device__ __forceinline__ float scale() const { return n * kHalfInv; }
 };
 
 template <int P, int RECON>
@@ -592,6 +636,18 @@ struct RawLink {
             h.decode(raw);
         }
         LinkIO<P, RECON>::reconstruct(raw, u);
+    }
+    // half, recon 18/12: the link in units of kHalfInv (the stored integers; the two-row
+    // reconstruction's third row, quadratic in them, is brought back to the same units)
+    __device__ __forceinline__ void decode_q(Cx<R> u[3][3]) const {
+        static_assert(P == 2 && RECON != 8, "deferred-scale decode: half recon 18/12 only");
+        R raw[RECON];
+        h.decode_q(raw);
+        LinkIO<P, RECON>::reconstruct(raw, u);
+        if constexpr (RECON == 12) {
+#pragma unroll
+            for (int c = 0; c < 3; ++c) u[2][c] = kHalfInv * u[2][c];
+        }
     }
 };
 

@@ -103,9 +103,11 @@ __device__ __forceinline__ void spatial_project(const Cx<R> p[4][3], Cx<R> h0[3]
         }
     }
 }
-template <int MU, int SIGMA, bool ADJ, typename R>
+// SC (deferred-scale half precision): h and u hold the stored integers, the hop result is
+// c * (U h) — the scale rides on the expansion's FFMA2s instead of one FMUL2 per decoded pair
+template <int MU, int SIGMA, bool ADJ, bool SC = false, typename R>
 __device__ __forceinline__ void spatial_mult_expand(const Cx<R> h0[3], const Cx<R> h1[3], const Cx<R> u[3][3],
-                                                    Cx<R> acc[4][3]) {
+                                                    Cx<R> acc[4][3], R c = (R)1) {
     Cx<R> g0[3], g1[3];
     if constexpr (ADJ) {
         su3_dag_mul(u, h0, g0);
@@ -113,6 +115,28 @@ __device__ __forceinline__ void spatial_mult_expand(const Cx<R> h0[3], const Cx<
     } else {
         su3_mul(u, h0, g0);
         su3_mul(u, h1, g1);
+    }
+    if constexpr (SC) {
+        static_assert(sizeof(R) == 4, "deferred scale: fp32 arithmetic only");
+        const float2 cc = bc(c), pc = make_float2(-c, c);  // acc + c g, acc + i c g
+        const float2 ps = SIGMA > 0 ? pc : make_float2(c, -c);
+#pragma unroll
+        for (int k = 0; k < 3; ++k) {
+            acc[0][k] = cf(__ffma2_rn(cc, f2(g0[k]), f2(acc[0][k])));
+            acc[1][k] = cf(__ffma2_rn(cc, f2(g1[k]), f2(acc[1][k])));
+            const float2 s0 = make_float2(g0[k].i, g0[k].r), s1 = make_float2(g1[k].i, g1[k].r);
+            if constexpr (MU == 0) {  // r2 = s i h1, r3 = s i h0
+                acc[2][k] = cf(__ffma2_rn(s1, ps, f2(acc[2][k])));
+                acc[3][k] = cf(__ffma2_rn(s0, ps, f2(acc[3][k])));
+            } else if constexpr (MU == 1) {  // r2 = -s h1, r3 = s h0
+                acc[2][k] = cf(__ffma2_rn(bc(SIGMA > 0 ? -c : c), f2(g1[k]), f2(acc[2][k])));
+                acc[3][k] = cf(__ffma2_rn(bc(SIGMA > 0 ? c : -c), f2(g0[k]), f2(acc[3][k])));
+            } else {  // r2 = s i h0, r3 = -s i h1
+                acc[2][k] = cf(__ffma2_rn(s0, ps, f2(acc[2][k])));
+                acc[3][k] = cf(__ffma2_rn(s1, make_float2(-ps.x, -ps.y), f2(acc[3][k])));
+            }
+        }
+        return;
     }
 #pragma unroll
     for (int c = 0; c < 3; ++c) {
@@ -130,11 +154,43 @@ __device__ __forceinline__ void spatial_mult_expand(const Cx<R> h0[3], const Cx<
         }
     }
 }
-template <int MU, int SIGMA, bool ADJ, typename R>
-__device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3][3], Cx<R> acc[4][3]) {
+template <int MU, int SIGMA, bool ADJ, bool SC = false, typename R>
+__device__ __forceinline__ void spatial_hop(const Cx<R> p[4][3], const Cx<R> u[3][3], Cx<R> acc[4][3], R c = (R)1) {
     Cx<R> h0[3], h1[3];
     spatial_project<MU, SIGMA>(p, h0, h1);
-    spatial_mult_expand<MU, SIGMA, ADJ>(h0, h1, u, acc);
+    spatial_mult_expand<MU, SIGMA, ADJ, SC>(h0, h1, u, acc, c);
+}
+
+// Decoding with or without the deferred scale (DF): returns the factor the values carry
+template <bool DF, int P, int N>
+__device__ __forceinline__ typename Prec<P>::R dec_vec(const RawVec<P, N> &r, typename Prec<P>::R *out) {
+    if constexpr (DF) {
+        r.decode_q(out);
+        return r.scale();
+    } else {
+        r.decode(out);
+        return (typename Prec<P>::R)1;
+    }
+}
+template <bool DF, int P, int RECON>
+__device__ __forceinline__ typename Prec<P>::R dec_link(const RawLink<P, RECON> &l, Cx<typename Prec<P>::R> u[3][3]) {
+    if constexpr (DF) {
+        l.decode_q(u);
+        return kHalfInv;
+    } else {
+        l.decode(u);
+        return (typename Prec<P>::R)1;
+    }
+}
+// whether the half-precision Dslash defers the decode scale (recon 8 reconstructs through
+// sqrt/sincos of the true values, so it keeps the scaled decode).  QX_NO_DEFER: A/B builds.
+template <int P, int RECON>
+__host__ __device__ constexpr bool dslash_defer() {
+#ifdef QX_NO_DEFER
+    return false;
+#else
+    return P == 2 && RECON != 8;
+#endif
 }
 
 // Faces of a partitioned X / Y / Z: the projected half spinor (h0, h1), 12 reals in the
@@ -188,20 +244,22 @@ struct SFace {
 // spin projection (SFace).  Half: the sender's raw 16-bit record (same layout as a half spinor
 // field with stride fs, norm included; 52 B per site, less than a projected fp32 face) projected
 // here from exactly the values the unpartitioned kernel decodes.
-template <int P, int MU, int SIGMA>
-__device__ __forceinline__ void ghost_half(const void *base, long fs, long f, Cx<typename Prec<P>::R> h0[3],
-                                           Cx<typename Prec<P>::R> h1[3]) {
+template <int P, int MU, int SIGMA, bool DF>
+__device__ __forceinline__ typename Prec<P>::R ghost_half(const void *base, long fs, long f, Cx<typename Prec<P>::R> h0[3],
+                                                          Cx<typename Prec<P>::R> h1[3]) {
     using R = typename Prec<P>::R;
     if constexpr (P == 2) {
         RawVec<2, 24> sv;
         sv.template load_spinor<0>(base, fs, f);
         R v[24];
         Cx<R> ps[4][3];
-        sv.decode(v);
+        const R sc = dec_vec<DF>(sv, v);
         unpack_spinor(v, ps);
         spatial_project<MU, SIGMA>(ps, h0, h1);
+        return sc;
     } else {
         SFace<R>::load(base, fs, f, h0, h1);
+        return (R)1;
     }
 }
 // index of a site in the face of dimension mu (lexicographic over the other three local
@@ -278,13 +336,16 @@ __device__ __forceinline__ void herm6_mul(const R *m, const Cx<R> v[6], Cx<R> ou
 template <int P>
 struct CloverIO {
     using R = typename Prec<P>::R;
-    // chiral block b (0: C+, 1: C-) of site i: 36 reals
-    static __device__ __forceinline__ void load(const void *base, long stride, long i, int b, R *m) {
+    // chiral block b (0: C+, 1: C-) of site i: 36 reals.  DF (half): the stored integers, the
+    // returned block scale to be applied to the product (deferred-scale decode)
+    template <bool DF = false>
+    static __device__ __forceinline__ R load(const void *base, long stride, long i, int b, R *m) {
         if constexpr (P == 8) {
             Blocks<8, 18, true>::load(base, stride, i, 18 * b, m);
         } else if constexpr (P == 4) {
             Blocks<4, 9, true>::load(base, stride, i, 9 * b, m);
         } else {
+            static_assert(P == 2 || !DF, "deferred clover scale: half only");
             // 9 uint4 regions (reals 8k..8k+7); chiral block b = reals 36b..36b+35, so region 4
             // is split: its low 8 bytes end C+, its high 8 bytes start C-
             const float2 nn = ld_stream(reinterpret_cast<const float2 *>(cptr(base, (size_t)144 * stride)) + i);
@@ -302,11 +363,13 @@ struct CloverIO {
             q[b ? 1 : 17] = mid.y;
 #pragma unroll
             for (int k = 0; k < 18; ++k) {
-                const float2 d = dq2(q[k], scale);
+                const float2 d = DF ? dq2_q(q[k]) : dq2(q[k], scale);
                 m[2 * k] = d.x;
                 m[2 * k + 1] = d.y;
             }
+            return DF ? scale : 1.f;
         }
+        return (R)1;
     }
 };
 
@@ -322,14 +385,23 @@ __device__ __forceinline__ void apply_clover(const void *cl, long stride, long i
             va[s * 3 + c] = in[s][c] + in[s + 2][c];
             vb[s * 3 + c] = in[s][c] - in[s + 2][c];
         }
+    constexpr bool DF = (P == 2) && dslash_defer<2, 12>();
     {
         R m[36];
-        CloverIO<P>::load(cl, stride, i, 0, m);
+        const R sc = CloverIO<P>::template load<DF>(cl, stride, i, 0, m);
+        if constexpr (DF) {
+#pragma unroll
+            for (int k = 0; k < 6; ++k) va[k] = sc * va[k];
+        }
         herm6_mul(m, va, wa);
     }
     {
         R m[36];
-        CloverIO<P>::load(cl, stride, i, 1, m);
+        const R sc = CloverIO<P>::template load<DF>(cl, stride, i, 1, m);
+        if constexpr (DF) {
+#pragma unroll
+            for (int k = 0; k < 6; ++k) vb[k] = sc * vb[k];
+        }
         herm6_mul(m, vb, wb);
     }
 #pragma unroll
@@ -438,6 +510,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // of the backward hop are issued before the forward hop is computed: twice the bytes in
     // flight per thread (dslash_pair).
     constexpr bool PAIR = dslash_pair<P, RECON>();
+    constexpr bool DF = dslash_defer<P, RECON>();
     auto spatial = [&](auto mu_c, int coord, int Lmu, int nf, int nb) {
         constexpr int MU = decltype(mu_c)::value;
         if (SS && ((a.smask >> MU) & 1)) {
@@ -446,41 +519,42 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             if (gf || gb) {
                 const int f = face_index<MU>(x, y, z, t, X, Y, Z);
                 Cx<R> h0[3], h1[3], u[3][3];
+                R sc;
                 if (gf) {
-                    ghost_half<P, MU, SF>(a.sghost_fwd[MU], a.sfs[MU], f, h0, h1);
+                    sc = ghost_half<P, MU, SF, DF>(a.sghost_fwd[MU], a.sfs[MU], f, h0, h1);
                 } else {
                     RawVec<P, 24> sv;
                     sv.template load_spinor<INMODE>(fin, a.stride, nf);
                     R v[24];
                     Cx<R> ps[4][3];
-                    sv.decode(v);
+                    sc = dec_vec<DF>(sv, v);
                     unpack_spinor(v, ps);
                     spatial_project<MU, SF>(ps, h0, h1);
                 }
                 {
                     RawLink<P, RECON> l;
                     l.load(a.gauge[MU][p], a.stride, i);
-                    l.decode(u);
+                    sc *= dec_link<DF>(l, u);
                 }
-                spatial_mult_expand<MU, SF, false>(h0, h1, u, acc);
+                spatial_mult_expand<MU, SF, false, DF>(h0, h1, u, acc, sc);
                 if (gb) {
-                    ghost_half<P, MU, SB>(a.sghost_back[MU], a.sfs[MU], f, h0, h1);
+                    sc = ghost_half<P, MU, SB, DF>(a.sghost_back[MU], a.sfs[MU], f, h0, h1);
                     RawLink<P, RECON> l;
                     l.load(a.gauge_sghost[MU], a.sfs[MU], f);
-                    l.decode(u);
+                    sc *= dec_link<DF>(l, u);
                 } else {
                     RawVec<P, 24> sv;
                     sv.template load_spinor<INMODE>(fin, a.stride, nb);
                     R v[24];
                     Cx<R> ps[4][3];
-                    sv.decode(v);
+                    sc = dec_vec<DF>(sv, v);
                     unpack_spinor(v, ps);
                     spatial_project<MU, SB>(ps, h0, h1);
                     RawLink<P, RECON> l;
                     l.load(a.gauge[MU][op], a.stride, nb);
-                    l.decode(u);
+                    sc *= dec_link<DF>(l, u);
                 }
-                spatial_mult_expand<MU, SB, true>(h0, h1, u, acc);
+                spatial_mult_expand<MU, SB, true, DF>(h0, h1, u, acc, sc);
                 return;
             }
         }
@@ -495,10 +569,10 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         {
             R v[24];
             Cx<R> ps[4][3], u[3][3];
-            sf.decode(v);
+            R sc = dec_vec<DF>(sf, v);
             unpack_spinor(v, ps);
-            lf.decode(u);
-            spatial_hop<MU, SF, false>(ps, u, acc);
+            sc *= dec_link<DF>(lf, u);
+            spatial_hop<MU, SF, false, DF>(ps, u, acc, sc);
         }
         if constexpr (!PAIR) {
             sb.template load_spinor<INMODE>(fin, a.stride, nb);
@@ -507,10 +581,10 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         {
             R v[24];
             Cx<R> ps[4][3], u[3][3];
-            sb.decode(v);
+            R sc = dec_vec<DF>(sb, v);
             unpack_spinor(v, ps);
-            lb.decode(u);
-            spatial_hop<MU, SB, true>(ps, u, acc);
+            sc *= dec_link<DF>(lb, u);
+            spatial_hop<MU, SB, true, DF>(ps, u, acc, sc);
         }
     };
     spatial(std::integral_constant<int, 0>{}, x, X, (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1,
@@ -555,17 +629,17 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         {
             R h[12];
             Cx<R> u[3][3];
-            hf.decode(h);
-            lf.decode(u);
-            temporal_hop<FWD_UPPER, false>(h, u, cf, acc);
+            R sc = dec_vec<DF>(hf, h);
+            sc *= dec_link<DF>(lf, u);
+            temporal_hop<FWD_UPPER, false>(h, u, DF ? cf * sc : cf, acc);
         }
         if constexpr (!PAIR) load_b();
         {
             R h[12];
             Cx<R> u[3][3];
-            hb.decode(h);
-            lb.decode(u);
-            temporal_hop<BWD_UPPER, true>(h, u, cb, acc);
+            R sc = dec_vec<DF>(hb, h);
+            sc *= dec_link<DF>(lb, u);
+            temporal_hop<BWD_UPPER, true>(h, u, DF ? cb * sc : cb, acc);
         }
     }
 

@@ -1,6 +1,8 @@
 """Cost of the split (halo) Dslash path at N=1: Mhat through the unsplit kernel vs the NCCL
 loopback (pack -> send/recv to self -> interior + boundary) vs the kernel-initiated P2P
-loopback (pack stores into the ghosts + flag release -> interior + boundary acquire).
+loopback (pack stores into the ghosts + flag release -> interior + boundary acquire), and the
+multi-dimensional split in loopback (Z, Z+T, Y+Z+T, all four: projected X/Y/Z faces, interior
+box + boundary-list kernels).
 
     python scripts/bench_halo.py [--dims 32,32,32,64] [--reps 50] [--prec 4]
 """
@@ -29,6 +31,9 @@ def main():
     res = {"dims": dims, "prec": args.prec}
     modes = (("unsplit", {}), ("nccl_loopback", {"comm": qudax.COMM_NCCL, "nccl_id": qudax.nccl_unique_id()}),
              ("p2p_loopback", {"halo": qudax.HALO_P2P}))
+    nid = qudax.nccl_unique_id
+    modes += tuple((f"nccl_loopback_split{m:04b}", {"comm": qudax.COMM_NCCL, "nccl_id": nid(), "split_mask": m})
+                   for m in (0b0100, 0b1100, 0b1110, 0b1111))
     for name, kw in modes:
         ctx = qudax.Context(dims, **kw)
         ctx.gauge_load(U, 0.124, 1.0, prec=args.prec, recon=12 if args.prec != 8 else 18)
