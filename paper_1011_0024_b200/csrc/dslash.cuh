@@ -513,8 +513,25 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     constexpr bool DF = dslash_defer<P, RECON>();
     auto spatial = [&](auto mu_c, int coord, int Lmu, int nf, int nb) {
         constexpr int MU = decltype(mu_c)::value;
-        if (SS && ((a.smask >> MU) & 1)) {
-            // partitioned dimension: a hop off the local box reads the neighbour's projected face
+        // operand sources of the two hops: the input field, or (partitioned X) the neighbour's
+        // raw face records — a per-lane pointer select, so the warps (every one of which holds
+        // x = 0 / x = X-1 sites) do not diverge
+        const void *fsrc = fin, *bsrc = fin, *lbsrc = a.gauge[MU][op];
+        long fstr = a.stride, bstr = a.stride, lbstr = a.stride;
+        int lbi = nb;
+        if constexpr (SS && MU == 0) {
+            if (a.smask & 1) {
+                const int f = face_index<0>(x, y, z, t, X, Y, Z);
+                if (coord == Lmu - 1) { fsrc = a.sghost_fwd[0]; fstr = a.sfs[0]; nf = f; }
+                if (coord == 0) {
+                    bsrc = a.sghost_back[0]; bstr = a.sfs[0]; nb = f;
+                    lbsrc = a.gauge_sghost[0]; lbstr = a.sfs[0]; lbi = f;
+                }
+            }
+        }
+        if (SS && MU > 0 && ((a.smask >> MU) & 1)) {
+            // partitioned Y / Z: a hop off the local box reads the neighbour's projected face
+            // (whole rows / planes: no divergence)
             const bool gf = (coord == Lmu - 1), gb = (coord == 0);
             if (gf || gb) {
                 const int f = face_index<MU>(x, y, z, t, X, Y, Z);
@@ -560,11 +577,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         }
         RawVec<P, 24> sf, sb;
         RawLink<P, RECON> lf, lb;
-        sf.template load_spinor<INMODE>(fin, a.stride, nf);
+        sf.template load_spinor<INMODE>(fsrc, fstr, nf);
         lf.load(a.gauge[MU][p], a.stride, i);
         if constexpr (PAIR) {
-            sb.template load_spinor<INMODE>(fin, a.stride, nb);
-            lb.load(a.gauge[MU][op], a.stride, nb);
+            sb.template load_spinor<INMODE>(bsrc, bstr, nb);
+            lb.load(lbsrc, lbstr, lbi);
         }
         {
             R v[24];
@@ -575,8 +592,8 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             spatial_hop<MU, SF, false, DF>(ps, u, acc, sc);
         }
         if constexpr (!PAIR) {
-            sb.template load_spinor<INMODE>(fin, a.stride, nb);
-            lb.load(a.gauge[MU][op], a.stride, nb);
+            sb.template load_spinor<INMODE>(bsrc, bstr, nb);
+            lb.load(lbsrc, lbstr, lbi);
         }
         {
             R v[24];

@@ -186,8 +186,11 @@ int dslash_blocks_f16(int recon, int dagger, int kind, int nthreads);
 // face with its backward-hop projector -> sf[mu]; 12 reals per site in the arithmetic precision
 void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, const void *in, void *const sb[3],
                          void *const sf[3], cudaStream_t s);
+// whether the faces along mu carry raw spinor records (half everywhere; X in every precision)
+// instead of spin-projected half spinors in the arithmetic precision
+__host__ __device__ inline bool sface_raw(int prec, int mu) { return prec == 2 || mu == 0; }
 // bytes of one spatial face buffer along mu
-size_t sface_bytes(int prec, long fs);
+size_t sface_bytes(int prec, int mu, long fs);
 // face pack: t_loc = 0 slice half (lower if !dagger) -> send_back; t_loc = T_loc-1 half
 // (upper if !dagger) -> send_fwd.  `in` is the Dslash input field (parity 1-p).
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back,

@@ -644,7 +644,9 @@ void launch_pack_faces_p2p(int prec, int dagger, const Geom &g, const void *in, 
 // bit-identically to the unpartitioned kernel.  Half precision ships the raw 16-bit record and
 // its norm instead (52 B per site vs 48 B projected in fp32); the receiver projects it
 // (dslash.cuh ghost_half) — measured: a projected half face differed from the unsplit kernel
-// by one half-precision quantum on ~4% of the Y-face sites.
+// by one half-precision quantum on ~4% of the Y-face sites.  X faces are raw in every precision:
+// the receiver reads them through the ordinary hop with a per-lane pointer select (x = 0 and
+// x = X-1 sites sit in every warp, so a separate ghost branch would diverge everywhere).
 struct SPackArgs {
     int L[4];
     int mask;       // split spatial dims
@@ -669,14 +671,21 @@ __global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *
     face_site(mu, f, fwd ? a.L[mu] - 1 : 0, a.q, a.L, c);
     const long i = (((long)(c[3] * a.L[2] + c[2]) * a.L[1] + c[1]) * a.L[0] + c[0]) >> 1;
     void *dst = fwd ? a.sf[mu] : a.sb[mu];
-    if constexpr (P == 2) {  // half: the raw record + norm (bits only; the receiver projects)
-        for (int hf = 0; hf < 2; ++hf) {
-            reinterpret_cast<uint4 *>(mptr(dst, h_spinor_u(a.fsd[mu], hf)))[f] =
-                reinterpret_cast<const uint4 *>(cptr(in, h_spinor_u(a.stride, hf)))[i];
-            reinterpret_cast<uint2 *>(mptr(dst, h_spinor_v(a.fsd[mu], hf)))[f] =
-                reinterpret_cast<const uint2 *>(cptr(in, h_spinor_v(a.stride, hf)))[i];
+    if (sface_raw(P, mu)) {  // the raw record (+ half norm): bits only, the receiver projects
+        if constexpr (P == 2) {
+            for (int hf = 0; hf < 2; ++hf) {
+                reinterpret_cast<uint4 *>(mptr(dst, h_spinor_u(a.fsd[mu], hf)))[f] =
+                    reinterpret_cast<const uint4 *>(cptr(in, h_spinor_u(a.stride, hf)))[i];
+                reinterpret_cast<uint2 *>(mptr(dst, h_spinor_v(a.fsd[mu], hf)))[f] =
+                    reinterpret_cast<const uint2 *>(cptr(in, h_spinor_v(a.stride, hf)))[i];
+            }
+            SpinorIO<2>::norms(dst, a.fsd[mu])[f] = SpinorIO<2>::norms(in, a.stride)[i];
+        } else {
+            using V = typename StoreVec<P>::V;
+            constexpr int NB = (P == 8) ? 12 : 6;
+            for (int b = 0; b < NB; ++b)
+                reinterpret_cast<V *>(dst)[b * a.fsd[mu] + f] = reinterpret_cast<const V *>(in)[b * a.stride + i];
         }
-        SpinorIO<2>::norms(dst, a.fsd[mu])[f] = SpinorIO<2>::norms(in, a.stride)[i];
         return;
     }
     RawVec<P, 24> raw;
@@ -696,7 +705,7 @@ __global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *
     SFace<R>::store(dst, a.fsd[mu], f, h0, h1);
 }
 
-size_t sface_bytes(int prec, long fs) { return prec == 2 ? spinor_bytes(2, fs) : (size_t)12 * prec * fs; }
+size_t sface_bytes(int prec, int mu, long fs) { return sface_raw(prec, mu) ? spinor_bytes(prec, fs) : (size_t)12 * prec * fs; }
 
 void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, const void *in, void *const sb[3],
                          void *const sf[3], cudaStream_t s) {

@@ -24,6 +24,7 @@ def main():
     ap.add_argument("--dims", default="32,32,32,64")
     ap.add_argument("--reps", type=int, default=50)
     ap.add_argument("--prec", type=int, default=4)
+    ap.add_argument("--modes", default="", help="comma list of mode names to run (default all)")
     args = ap.parse_args()
     dims = tuple(int(v) for v in args.dims.split(","))
     U = qgen.gauge(dims, 1005, eps=0.1)
@@ -33,7 +34,9 @@ def main():
              ("p2p_loopback", {"halo": qudax.HALO_P2P}))
     nid = qudax.nccl_unique_id
     modes += tuple((f"nccl_loopback_split{m:04b}", {"comm": qudax.COMM_NCCL, "nccl_id": nid(), "split_mask": m})
-                   for m in (0b0100, 0b1100, 0b1110, 0b1111))
+                   for m in (0b0001, 0b0100, 0b1100, 0b1110, 0b1111))
+    if args.modes:
+        modes = tuple(m for m in modes if m[0] in args.modes.split(","))
     for name, kw in modes:
         ctx = qudax.Context(dims, **kw)
         ctx.gauge_load(U, 0.124, 1.0, prec=args.prec, recon=12 if args.prec != 8 else 18)
