@@ -204,6 +204,10 @@ def config3_solve_time():
     res = {"workload": "24^3x128 weak field, 6 point sources, tol 1e-14, kappa 0.124, csw 1.0 (BASELINE configs[2])"}
     for name, ps, delta in (("double-single", 4, 0.1), ("double-half", 2, 0.1)):
         ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=ps, recon_sloppy=12, t_boundary=-1)
+        srcs = [qgen.point_source(dims, spin, colour) for colour in range(3) for spin in range(2)]
+        # warm-up (workspace allocation, graph capture) outside the timed solves, for both forms
+        ctx.solve(srcs[0], tol=0, delta=delta, maxiter=3, prec=8, prec_sloppy=ps, allow_not_converged=True)
+        ctx.solve_multi(srcs, tol=0, delta=delta, maxiter=3, prec=8, prec_sloppy=ps, allow_not_converged=True)
         ts, its, trs, gfl = [], [], [], []
         for colour in range(3):
             for spin in range(2):
@@ -216,6 +220,15 @@ def config3_solve_time():
                 gfl.append(st["gflops"])
         res[name] = {"mean_secs": sum(ts) / len(ts), "mean_iters": sum(its) / len(its), "max_true_res": max(trs),
                      "mean_gflops": sum(gfl) / len(gfl)}
+        # the same 6 sources as ONE batched solve (multi-RHS Mhat, per-system fused reductions):
+        # seconds per source = batch wall time / 6
+        _, sts = ctx.solve_multi(srcs, tol=1e-14, delta=delta, maxiter=20000, prec=8, prec_sloppy=ps,
+                                 allow_not_converged=True)
+        secs = sts[0]["secs"]
+        res[name + " batched x6"] = {"secs_per_source": secs / len(srcs), "batch_secs": secs,
+                                     "mean_iters": sum(s["iters"] for s in sts) / len(sts),
+                                     "max_true_res": max(s["true_res"] for s in sts),
+                                     "gflops": sum(s["flops"] for s in sts) / secs * 1e-9}
     ctx.close()
     return res
 

@@ -314,6 +314,20 @@ qudax_status qudax_solve_bicgstab(qudax_ctx *ctx, double *host_x, const double *
 qudax_status qudax_solve_bicgstab_dev(qudax_ctx *ctx, double *dev_x, const double *dev_b,
                                       const qudax_solve_param *p, qudax_solve_stats *st);
 
+/* Batched mixed-precision BiCGstab for nrhs (1..8) sources on the same gauge field (SURVEY 8(f)
+ * item 2; the paper solves 6 sources per configuration).  Every system runs its own
+ * Algorithm R — iterates, reliable updates and the returned x are exactly those of nrhs calls of
+ * qudax_solve_bicgstab on an unpartitioned context — but each iteration applies Mhat to all
+ * still-active systems with one multi-RHS kernel pair, the <rhat0, v> and (<t, s>, |t|^2)
+ * reductions fused per system into its epilogue.  use_schur 0 or 1 (asymmetric form); the
+ * residual history, if requested, is that of system 0.  host_x / host_b: arrays of nrhs full
+ * local slabs (as qudax_solve_bicgstab); st: nrhs stats (secs = the batch's wall time).
+ * Returns QUDAX_ERR_NOT_CONVERGED if any system missed tol. */
+qudax_status qudax_solve_bicgstab_multi(qudax_ctx *ctx, double *const *host_x, const double *const *host_b, int nrhs,
+                                        const qudax_solve_param *p, qudax_solve_stats *st);
+qudax_status qudax_solve_bicgstab_multi_dev(qudax_ctx *ctx, double *const *dev_x, const double *const *dev_b,
+                                            int nrhs, const qudax_solve_param *p, qudax_solve_stats *st);
+
 /* CGNR ("Conjugate Gradients [7] on the normal equations"): CG on
  * Mhat^dag Mhat x_e = Mhat^dag bhat in precision p->prec (prec_sloppy and delta ignored), with
  * the same Schur prepare / reconstruct and the same TRUE-residual stopping test as BiCGstab. */

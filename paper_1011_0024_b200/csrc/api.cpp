@@ -560,7 +560,7 @@ void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, con
 // different RHS so the links and clover are read from HBM about once for all of them.
 // Partitioned runs (halo exchange per RHS) apply the single-RHS path per field.
 void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, const void *const *x, int n, int prec,
-                     int p, int dagger, int kind, double a, int reverse) {
+                     int p, int dagger, int kind, double a, int reverse, const RedReq *reds) {
     check_prec(prec);
     QX_CHECK(n >= 1 && n <= kMaxRhs, QUDAX_ERR_ARG, "nrhs must be 1.." + std::to_string(kMaxRhs));
     QX_CHECK(p == 0 || p == 1, QUDAX_ERR_ARG, "parity must be 0 or 1");
@@ -571,7 +571,7 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
     }
     if (c->comm != QUDAX_COMM_NONE || c->p2p.on || n == 1) {
         for (int k = 0; k < n; ++k)
-            dslash_op(c, out[k], in[k], x ? x[k] : nullptr, prec, p, dagger, kind, a, nullptr, reverse);
+            dslash_op(c, out[k], in[k], x ? x[k] : nullptr, prec, p, dagger, kind, a, reds ? reds + k : nullptr, reverse);
         return;
     }
     auto &gc = gauge_for(c, prec);
@@ -582,6 +582,26 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
         args.out_m[k] = out[k];
         args.x_m[k] = x ? x[k] : nullptr;
     }
+    if (reds) {  // one deterministic reduction (and scalar recurrence) per right-hand side
+        const Geom &g = c->g;
+        const int nb = dslash_blocks_any(prec, gc.recon, dagger, kind, (int)g.Vh);
+        const size_t slots = 3 * ((size_t)nb + nb / kGroupHost + 2);
+        const size_t ncount = 2 + (size_t)nb / kGroupHost + 2;
+        if (!c->dpart_m) {
+            c->dpart_m = static_cast<double *>(dalloc(c, sizeof(double) * slots * kMaxRhs));
+            c->dcount_m = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * ncount * kMaxRhs));
+            QX_CUDA(cudaMemsetAsync(c->dcount_m, 0, sizeof(unsigned) * ncount * kMaxRhs, c->stream));
+        }
+        args.red_kind = reds[0].kind;
+        for (int k = 0; k < n; ++k) {
+            QX_CHECK(reds[k].kind == reds[0].kind && reds[k].S, QUDAX_ERR_ARG, "multi-RHS reductions: one kind, device scalars");
+            QX_CHECK(reds[k].kind != RED_XDOT_NORM || kind >= QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
+            QX_CHECK(reds[k].kind != RED_RHAT_DOT || reds[k].rhat, QUDAX_ERR_ARG, "rhat-dot needs rhat");
+            args.rhat_m[k] = reds[k].rhat;
+            args.tail_m[k] = RedTail{c->dpart_m + slots * k, c->dcount_m + ncount * k, nb, 0, reds[k].S->red, reds[k].S,
+                                     reds[k].coef_mode};
+        }
+    }
     args.ghosted = 0;
     args.range = RANGE_ALL;
     args.nthreads = (int)c->g.Vh;
@@ -589,7 +609,8 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
     c->launches += 1;
 }
 
-void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger) {
+void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger,
+                    const RedReq *reds) {
     QX_CHECK(n >= 1 && n <= kMaxRhs, QUDAX_ERR_ARG, "nrhs must be 1.." + std::to_string(kMaxRhs));
     void *t[kMaxRhs];
     for (int k = 0; k < n; ++k) {
@@ -597,8 +618,9 @@ void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n
         if (!slot) slot = dalloc(c, spinor_bytes(prec, c->g.stride));
         t[k] = slot;
     }
-    dslash_multi_op(c, t, in, nullptr, n, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, 0);
-    dslash_multi_op(c, out, t, in, n, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, 1);
+    QX_CHECK(!c->matpc_sym, QUDAX_ERR_UNSUPPORTED, "multi-RHS Mhat: asymmetric Schur form only");
+    dslash_multi_op(c, t, in, nullptr, n, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, 0, nullptr);
+    dslash_multi_op(c, out, t, in, n, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, 1, reds);
 }
 
 void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int parity, bool inverse) {
@@ -1414,9 +1436,63 @@ qudax_status solve_host_entry(SolveFn fn, qudax_ctx *c, double *host_x, const do
     if (s == QUDAX_OK && p->tol > 0 && st->true_res > p->tol * (1 + 1e-3)) return QUDAX_ERR_NOT_CONVERGED;
     return s;
 }
+// batched solve: device slabs, or host slabs staged through the ctx (H2D / D2H inside)
+qudax_status solve_multi_entry(qudax_ctx *c, double *const *x, const double *const *b, int nrhs,
+                               const qudax_solve_param *p, qudax_solve_stats *st, bool host) {
+    if (!c) return QUDAX_ERR_ARG;
+    double *dbuf = nullptr;
+    auto t0 = std::chrono::steady_clock::now();
+    qudax_status s = guard(c, [&] {
+        QX_CHECK(x && b && p && st && nrhs >= 1 && nrhs <= kMaxRhs, QUDAX_ERR_ARG, "solve_multi: bad argument");
+        for (int j = 0; j < nrhs; ++j) QX_CHECK(x[j] && b[j], QUDAX_ERR_ARG, "solve_multi: null slab");
+        double *dx[kMaxRhs];
+        const double *db[kMaxRhs];
+        const size_t n = sizeof(double) * 24 * c->g.V;
+        if (host) {
+            dbuf = static_cast<double *>(dalloc(c, 2 * n * nrhs));
+            for (int j = 0; j < nrhs; ++j) {
+                db[j] = dbuf + (size_t)2 * j * (n / sizeof(double));
+                dx[j] = const_cast<double *>(db[j]) + n / sizeof(double);
+                QX_CUDA(cudaMemcpyAsync(const_cast<double *>(db[j]), b[j], n, cudaMemcpyHostToDevice, c->stream));
+            }
+        } else {
+            for (int j = 0; j < nrhs; ++j) {
+                db[j] = b[j];
+                dx[j] = x[j];
+            }
+        }
+        solve_multi_dev(c, dx, db, nrhs, p, st);
+        if (host) {
+            for (int j = 0; j < nrhs; ++j)
+                QX_CUDA(cudaMemcpyAsync(x[j], dx[j], n, cudaMemcpyDeviceToHost, c->stream));
+            QX_CUDA(cudaStreamSynchronize(c->stream));
+            dfree(c, dbuf);
+            dbuf = nullptr;
+        }
+        const double secs = std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
+        for (int j = 0; j < nrhs; ++j) {
+            st[j].secs = secs;  // the batch's wall time
+            st[j].gflops = st[j].flops / secs * 1e-9;
+        }
+    });
+    if (dbuf) { cudaStreamSynchronize(c->stream); dfree(c, dbuf); }
+    if (s == QUDAX_OK && p->tol > 0)
+        for (int j = 0; j < nrhs; ++j)
+            if (st[j].true_res > p->tol * (1 + 1e-3)) return QUDAX_ERR_NOT_CONVERGED;
+    return s;
+}
 }  // namespace
 
 extern "C" {
+
+qudax_status qudax_solve_bicgstab_multi(qudax_ctx *c, double *const *host_x, const double *const *host_b, int nrhs,
+                                        const qudax_solve_param *p, qudax_solve_stats *st) {
+    return solve_multi_entry(c, host_x, host_b, nrhs, p, st, true);
+}
+qudax_status qudax_solve_bicgstab_multi_dev(qudax_ctx *c, double *const *x, const double *const *b, int nrhs,
+                                            const qudax_solve_param *p, qudax_solve_stats *st) {
+    return solve_multi_entry(c, x, b, nrhs, p, st, false);
+}
 
 qudax_status qudax_solve_bicgstab_dev(qudax_ctx *c, double *x, const double *b, const qudax_solve_param *p,
                                       qudax_solve_stats *st) {

@@ -109,6 +109,8 @@ struct qudax_ctx {
     double *partials = nullptr, *red_out = nullptr, *h_red = nullptr;
     double *dpart = nullptr;  // per-CTA partials of Dslash-fused reductions
     unsigned *d_counter = nullptr;  // last-CTA counter of the stream-ordered reductions
+    double *dpart_m = nullptr;      // multi-RHS fused reductions: per-RHS CTA slots and counters
+    unsigned *dcount_m = nullptr;
     double *stage = nullptr;  // fp64 full-slab staging (V_loc * 24 doubles)
     int *d_flag = nullptr;
 
@@ -118,7 +120,8 @@ struct qudax_ctx {
         void *b_e = nullptr, *b_o = nullptr, *bh = nullptr, *x_e = nullptr, *x_o = nullptr, *r = nullptr, *t_e = nullptr,
              *t_o = nullptr;
         void *rs = nullptr, *xs = nullptr, *p = nullptr, *v = nullptr, *t = nullptr, *r0 = nullptr;
-    } sws, cgws;
+    } sws, cgws, mws[qx::kMaxRhs];
+    qx::SolverScalars *d_scal_m = nullptr, *h_scal_m = nullptr;  // batched solver: one set per RHS
 };
 
 namespace qx {
@@ -139,8 +142,11 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
 void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr);
 void matpc_sym_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr);
 void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, const void *const *x, int n, int prec,
-                     int p, int dagger, int kind, double a, int reverse);
-void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger);
+                     int p, int dagger, int kind, double a, int reverse, const RedReq *reds = nullptr);
+void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger,
+                    const RedReq *reds = nullptr);
+void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_dev, int n, const qudax_solve_param *p,
+                     qudax_solve_stats *st);
 int dslash_threads();
 void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int parity, bool inverse);
 // run a BLAS op; if it reduces, globally sum and return the values in res (host)

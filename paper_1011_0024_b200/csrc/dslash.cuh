@@ -708,7 +708,9 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // fused BiCGstab reductions over what was stored (half: the requantised values)
     SpinorIO<P>::store_requant(fout, a.stride, i, o);
     R w[24];
-    SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx : a.rhat, a.stride, i, w);
+    // (multi-RHS launch: this CTA's right-hand side, recomputed here rather than kept live)
+    const void *rh = a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat;
+    SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx : rh, a.stride, i, w);
 #pragma unroll
     for (int k = 0; k < 12; ++k) {
         const double orr = o[2 * k], oi = o[2 * k + 1], wr = w[2 * k], wi = w[2 * k + 1];
@@ -773,7 +775,10 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
             *a.p2p_cseq += 1u;
         }
     }
-    if (a.red_kind != RED_NONE) reduce_with_tail<3, QX_DSLASH_THREADS>(red, a.tail);
+    if (a.red_kind != RED_NONE) {
+        if (a.nrhs > 1) reduce_with_tail<3, QX_DSLASH_THREADS>(red, a.tail_m[blockIdx.x % a.nrhs], blockIdx.x / a.nrhs);
+        else reduce_with_tail<3, QX_DSLASH_THREADS>(red, a.tail);
+    }
 }
 
 template <int P, int RC, bool DG, int KD>

@@ -104,6 +104,7 @@ struct RedTail {
 // peers' face stores, the boundary fills the grid's tail)
 enum SiteRange { RANGE_ALL = 0, RANGE_INTERIOR = 1, RANGE_BOUNDARY = 2, RANGE_TAIL = 3 };
 constexpr int kMaxRhs = 8;
+constexpr int kGroupHost = 64;  // = reduce.cuh kGroup (slots per tail group)
 
 struct DslashArgs {
     // geometry
@@ -154,6 +155,10 @@ struct DslashArgs {
     const void *in_m[kMaxRhs];
     void *out_m[kMaxRhs];
     const void *x_m[kMaxRhs];
+    // fused reductions of a multi-RHS launch: one tail per right-hand side (the CTAs of one RHS
+    // form their own deterministic reduction; block index = site block)
+    const void *rhat_m[kMaxRhs];
+    RedTail tail_m[kMaxRhs];
 };
 enum DslashRed { RED_NONE = 0, RED_XDOT_NORM = 1, RED_RHAT_DOT = 2 };
 

@@ -14,6 +14,7 @@
 namespace qx {
 
 constexpr int kGroup = 64;
+static_assert(kGroup == kGroupHost, "host-side slot sizing (internal.h) must match");
 
 __device__ __forceinline__ double2 cdiv(double2 a, double2 b) {
     const double d = b.x * b.x + b.y * b.y;
@@ -69,11 +70,12 @@ __device__ __forceinline__ void cta_sum_slots(const double *src, int b0, int b1,
 // v[] -> this CTA's partial; the last CTA of the whole reduction produces t.out[0..NRED).
 // Layout: t.partials[0 .. total) CTA slots, then ceil(total/kGroup) group slots.
 // Counters: t.counter[0] groups done, t.counter[1 + g] CTAs done in group g (all zero on entry).
+// blk: this CTA's index within the reduction (-1: blockIdx.x)
 template <int NRED, int NT>
-__device__ __forceinline__ void reduce_with_tail(double (&v)[NRED], const RedTail &t) {
+__device__ __forceinline__ void reduce_with_tail(double (&v)[NRED], const RedTail &t, int blk = -1) {
     __shared__ double sm[NT / 32][NRED];
     __shared__ int stage;  // 0: not last in group; 1: last in group; 2: last overall
-    const int gb = t.block_offset + (int)blockIdx.x;
+    const int gb = t.block_offset + (blk < 0 ? (int)blockIdx.x : blk);
     const int ngroups = (t.total_blocks + kGroup - 1) / kGroup;
     const int grp = gb / kGroup;
     double *gslots = t.partials + (size_t)t.total_blocks * NRED;

@@ -23,6 +23,7 @@
 #include <complex>
 #include <cstdio>
 #include <cstring>
+#include <map>
 
 #include "ctx.h"
 
@@ -338,6 +339,206 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     st->flops = flops;
 }
 
+
+// Batched Algorithm R for n <= kMaxRhs right-hand sides ("multi-RHS Dslash /
+// block solver"; the paper's tests solve 6 sources per configuration, and production
+// calls the solver tens of thousands of times per configuration).  Each system
+// keeps its own Krylov space, scalars and reliable-update schedule — the iterates are exactly
+// those of n independent solve_dev calls — but the two Mhat applications of an iteration are
+// one multi-RHS launch pair for all still-active systems (links and clover streamed once for
+// all of them), with the <rhat0, v> and (<t, s>, |t|^2) reductions and scalar recurrences fused
+// per right-hand side into the second kernel.  A system leaves the batch when it converges.
+void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_dev, int n, const qudax_solve_param *sp,
+                     qudax_solve_stats *st) {
+    QX_CHECK(n >= 1 && n <= kMaxRhs, QUDAX_ERR_ARG, "nrhs must be 1.." + std::to_string(kMaxRhs));
+    QX_CHECK(sp->use_schur >= 0 && sp->use_schur <= 1, QUDAX_ERR_ARG, "multi-RHS solve: use_schur 0 or 1");
+    SchurForm form_guard(c, false);
+    QX_CHECK(c->gauge_loaded, QUDAX_ERR_STATE, "gauge not loaded");
+    const int Pd = sp->prec, Ps = sp->prec_sloppy;
+    check_prec(Pd);
+    check_prec(Ps);
+    QX_CHECK(sp->maxiter >= 0 && sp->tol >= 0 && sp->delta >= 0, QUDAX_ERR_ARG, "solve: bad parameters");
+    const Geom &g = c->g;
+    if (!c->d_scal_m) {
+        c->d_scal_m = static_cast<SolverScalars *>(dalloc(c, sizeof(SolverScalars) * kMaxRhs));
+        c->h_scal_m = static_cast<SolverScalars *>(halloc(c, sizeof(SolverScalars) * kMaxRhs));
+    }
+    struct Sys {
+        void *b_e, *b_o, *bh, *x_e, *x_o, *r, *t_e, *t_o, *rs, *xs, *p, *v, *t, *r0;
+        SolverScalars *S;
+        double bnorm, stop, rNorm, r0Norm, maxrr, maxrx, flops;
+        int k, updates, restarts;
+        bool converged, active;
+    } sys[kMaxRhs];
+    qudax_site_model mm;
+    qudax_model(4, 12, -1, &mm);
+    const double V_h_all = (double)g.Vh * g.nranks;
+    const double matpc_flops = mm.flops * V_h_all, blas_flops_iter = 960.0 * V_h_all;
+    for (int j = 0; j < n; ++j) {
+        auto &w = c->mws[j];
+        if (w.prec != Pd || w.prec_s != Ps) {
+            w = qudax_ctx::SolverWs{};
+            w.prec = Pd;
+            w.prec_s = Ps;
+        }
+        Sys &y = sys[j];
+        y.b_e = field(c, w.b_e, Pd); y.b_o = field(c, w.b_o, Pd); y.bh = field(c, w.bh, Pd);
+        y.x_e = field(c, w.x_e, Pd); y.x_o = field(c, w.x_o, Pd); y.r = field(c, w.r, Pd);
+        y.t_e = field(c, w.t_e, Pd); y.t_o = field(c, w.t_o, Pd);
+        y.rs = field(c, w.rs, Ps); y.xs = field(c, w.xs, Ps); y.p = field(c, w.p, Ps);
+        y.v = field(c, w.v, Ps); y.t = field(c, w.t, Ps); y.r0 = field(c, w.r0, Ps);
+        y.S = c->d_scal_m + j;
+        std::memset(&st[j], 0, sizeof(st[j]));
+        prepare_source(c, Pd, b_dev[j], y.b_e, y.b_o, y.bh, y.t_e, y.t_o, sp->use_schur);
+        y.bnorm = std::sqrt(norm2_of(c, Pd, y.bh));
+        y.stop = sp->tol * y.bnorm;
+        zero(c, y.x_e, Pd);
+        zero(c, y.xs, Ps);
+        zero(c, y.v, Ps);
+        zero(c, y.p, Ps);
+        copy(c, y.r, y.bh, Pd);
+        convert_op(c, y.rs, Ps, y.r, Pd);
+        copy(c, y.r0, y.rs, Ps);
+        y.rNorm = y.r0Norm = y.maxrr = y.maxrx = y.bnorm;
+        y.flops = 0;
+        y.k = y.updates = y.restarts = 0;
+        y.converged = (y.bnorm == 0.0);
+        y.active = !y.converged && sp->maxiter > 0;
+        SolverScalars h0{};
+        const cd rn = cdot_of(c, Ps, y.r0, y.rs);
+        h0.rho = make_double2(1, 0);
+        h0.rho_new = make_double2(rn.real(), rn.imag());
+        h0.alpha = make_double2(1, 0);
+        h0.omega = make_double2(1, 0);
+        QX_CUDA(cudaMemcpyAsync(y.S, &h0, sizeof(h0), cudaMemcpyHostToDevice, c->stream));
+    }
+    // one iteration of every active system; all scalars stay on the device
+    auto enqueue_iteration = [&](unsigned mask) {
+        void *vv[kMaxRhs], *pp[kMaxRhs], *tt[kMaxRhs], *ss[kMaxRhs];
+        RedReq red_rv[kMaxRhs], red_ts[kMaxRhs];
+        int na = 0;
+        for (int j = 0; j < n; ++j) {
+            if (!(mask >> j & 1)) continue;
+            Sys &y = sys[j];
+            void *f[3] = {y.rs, y.p, y.v};
+            CoefArg co[2] = {{{0, 0}, &y.S->beta}, {{0, 0}, &y.S->omega}};
+            blas_op_dev(c, OP_P_UPDATE, Ps, f, co, y.S, COEF_NONE);  // p = r + beta (p - omega v)
+            vv[na] = y.v; pp[na] = y.p; tt[na] = y.t; ss[na] = y.rs;
+            red_rv[na] = RedReq{RED_RHAT_DOT, y.r0, nullptr, y.S, COEF_ALPHA};
+            red_ts[na] = RedReq{RED_XDOT_NORM, nullptr, nullptr, y.S, COEF_OMEGA};
+            ++na;
+        }
+        matpc_multi_op(c, vv, pp, na, Ps, 0, red_rv);  // v = Mhat p; alpha = rho'/<rhat0, v>
+        for (int j = 0; j < n; ++j) {
+            if (!(mask >> j & 1)) continue;
+            void *f[2] = {sys[j].v, sys[j].rs};
+            CoefArg co[1] = {{{0, 0}, &sys[j].S->malpha}};
+            blas_op_dev(c, OP_CAXPY, Ps, f, co, sys[j].S, COEF_NONE);  // s = r - alpha v
+        }
+        matpc_multi_op(c, tt, ss, na, Ps, 0, red_ts);  // t = Mhat s; omega = <t,s>/|t|^2
+        for (int j = 0; j < n; ++j) {
+            if (!(mask >> j & 1)) continue;
+            Sys &y = sys[j];
+            void *f[5] = {y.xs, y.p, y.rs, y.t, y.r0};
+            CoefArg co[2] = {{{0, 0}, &y.S->alpha}, {{0, 0}, &y.S->omega}};
+            blas_op_dev(c, OP_FINAL, Ps, f, co, y.S, COEF_RHO);  // x += a p + w s; r = s - w t; rho', beta
+        }
+        QX_CUDA(cudaMemcpyAsync(c->h_scal_m, c->d_scal_m, sizeof(SolverScalars) * n, cudaMemcpyDeviceToHost, c->stream));
+    };
+    const bool use_graph = (c->comm != QUDAX_COMM_HOST) && !c->no_graphs && (c->g.nranks == 1 || c->force_graphs);
+    std::map<unsigned, std::pair<cudaGraphExec_t, long long>> graphs;  // one per active set
+    bool first = true;
+    for (;;) {
+        unsigned mask = 0;
+        for (int j = 0; j < n; ++j)
+            if (sys[j].active) mask |= 1u << j;
+        if (!mask) break;
+        if (!use_graph || first) {
+            enqueue_iteration(mask);  // the first iteration runs eagerly (lazily-created buffers)
+            first = false;
+        } else {
+            auto it = graphs.find(mask);
+            if (it == graphs.end()) {
+                long long nl = 0;
+                cudaGraphExec_t e = capture_graph(c, [&] { enqueue_iteration(mask); }, &nl);
+                it = graphs.emplace(mask, std::make_pair(e, nl)).first;
+            }
+            QX_CUDA(cudaGraphLaunch(it->second.first, c->stream));
+            c->launches += it->second.second;
+        }
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        harvest_graph_timing(c);
+        for (int j = 0; j < n; ++j) {
+            Sys &y = sys[j];
+            if (!y.active) continue;
+            const SolverScalars &hs = c->h_scal_m[j];
+            const double rNorm_it = std::sqrt(hs.r2);
+            const bool blown = !std::isfinite(rNorm_it) || rNorm_it > 1e2 * y.maxrr;  // reading R3
+            y.rNorm = rNorm_it;
+            ++y.k;
+            y.flops += 2 * matpc_flops + blas_flops_iter;
+            if (!blown) {
+                if (y.rNorm > y.maxrx) y.maxrx = y.rNorm;
+                if (y.rNorm > y.maxrr) y.maxrr = y.rNorm;
+            }
+            const bool updX = !blown && (y.rNorm < sp->delta * y.r0Norm) && (y.r0Norm <= y.maxrx);
+            const bool updR = blown || ((y.rNorm < sp->delta * y.maxrr) && (y.r0Norm <= y.maxrr)) || updX ||
+                              (y.rNorm <= y.stop) || (y.k == sp->maxiter);
+            if (updR) {  // reliable update of system j alone (single-RHS high-precision operator)
+                if (std::isfinite(rNorm_it)) xpy_mixed_op(c, Pd, Ps, y.xs, y.x_e);
+                zero(c, y.xs, Ps);
+                matpc_op(c, y.r, y.x_e, Pd, 0);
+                double r2;
+                {
+                    void *f[2] = {y.bh, y.r};
+                    blas_op(c, OP_BMR_NORM, Pd, f, nullptr, &r2);
+                }
+                y.flops += matpc_flops;
+                convert_op(c, y.rs, Ps, y.r, Pd);
+                y.rNorm = std::sqrt(r2);
+                y.maxrr = y.rNorm;
+                if (updX || blown) y.r0Norm = y.maxrx = y.rNorm;
+                SolverScalars upd = hs;
+                if (blown) {
+                    copy(c, y.r0, y.rs, Ps);
+                    zero(c, y.p, Ps);
+                    zero(c, y.v, Ps);
+                    const cd rn = cdot_of(c, Ps, y.r0, y.rs);
+                    upd.rho = make_double2(1, 0);
+                    upd.rho_new = make_double2(rn.real(), rn.imag());
+                    upd.alpha = make_double2(1, 0);
+                    upd.omega = make_double2(1, 0);
+                    upd.beta = make_double2(0, 0);
+                    ++y.restarts;
+                } else {
+                    const cd rn = cdot_of(c, Ps, y.r0, y.rs);
+                    const cd rho(hs.rho.x, hs.rho.y), al(hs.alpha.x, hs.alpha.y), om(hs.omega.x, hs.omega.y);
+                    const cd beta = (rn / rho) * (al / om);
+                    upd.rho_new = make_double2(rn.real(), rn.imag());
+                    upd.beta = make_double2(beta.real(), beta.imag());
+                }
+                QX_CUDA(cudaMemcpyAsync(y.S, &upd, sizeof(upd), cudaMemcpyHostToDevice, c->stream));
+                QX_CUDA(cudaStreamSynchronize(c->stream));
+                ++y.updates;
+                if (y.rNorm <= y.stop) y.converged = true;
+            }
+            if (y.converged || y.k >= sp->maxiter) y.active = false;
+            if (j == 0 && sp->res_history && y.k - 1 < sp->history_cap)
+                sp->res_history[y.k - 1] = y.bnorm > 0 ? y.rNorm / y.bnorm : 0.0;
+        }
+    }
+    for (auto &kv : graphs) cudaGraphExecDestroy(kv.second.first);
+    release_graph_timing(c);
+    for (int j = 0; j < n; ++j) {
+        Sys &y = sys[j];
+        st[j].iters = y.k;
+        st[j].reliable_updates = y.updates;
+        st[j].restarts = y.restarts;
+        st[j].true_res_schur = y.bnorm > 0 ? y.rNorm / y.bnorm : 0.0;
+        finish_solution(c, Pd, x_dev[j], y.b_e, y.b_o, y.x_e, y.x_o, y.t_e, y.t_o, sp->use_schur, &st[j]);
+        st[j].flops = y.flops;
+    }
+}
 
 // CGNR ("Conjugate Gradients on the normal equations"): CG on the Hermitian
 // positive-definite Mhat^dag Mhat x = Mhat^dag bhat, in precision sp->prec (no reliable

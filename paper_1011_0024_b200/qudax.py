@@ -139,6 +139,10 @@ SIGNATURES = {
     "qudax_cdot": ([_P, _P, _P, _I, _DP], _I),
     "qudax_solve_bicgstab": ([_P, _DP, _DP, ctypes.POINTER(SolveParam), ctypes.POINTER(SolveStats)], _I),
     "qudax_solve_bicgstab_dev": ([_P, _P, _P, ctypes.POINTER(SolveParam), ctypes.POINTER(SolveStats)], _I),
+    "qudax_solve_bicgstab_multi": ([_P, ctypes.POINTER(_P), ctypes.POINTER(_P), _I, ctypes.POINTER(SolveParam),
+                                    ctypes.POINTER(SolveStats)], _I),
+    "qudax_solve_bicgstab_multi_dev": ([_P, ctypes.POINTER(_P), ctypes.POINTER(_P), _I, ctypes.POINTER(SolveParam),
+                                        ctypes.POINTER(SolveStats)], _I),
     "qudax_solve_cgnr": ([_P, _DP, _DP, ctypes.POINTER(SolveParam), ctypes.POINTER(SolveStats)], _I),
     "qudax_solve_cgnr_dev": ([_P, _P, _P, ctypes.POINTER(SolveParam), ctypes.POINTER(SolveStats)], _I),
 }
@@ -449,6 +453,35 @@ class Context:
         if rc and not (allow_not_converged and rc == 6):
             self._check(rc)
         return x, st.as_dict()
+
+    def solve_multi(self, bs, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
+                    allow_not_converged=False, history=None, outs=None):
+        """Batched solve of len(bs) <= 8 sources (host arrays, full local slabs): one multi-RHS
+        Mhat kernel pair per iteration for all still-active systems.  Returns (xs, [stats])."""
+        bs = [np.ascontiguousarray(b, dtype=np.complex128) for b in bs]
+        xs = outs if outs is not None else [np.zeros_like(b) for b in bs]
+        n = len(bs)
+        bp = (_P * n)(*[b.ctypes.data for b in bs])
+        xp = (_P * n)(*[x.ctypes.data for x in xs])
+        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history)
+        st = (SolveStats * n)()
+        rc = lib().qudax_solve_bicgstab_multi(self._h, xp, bp, n, ctypes.byref(sp), st)
+        if rc and not (allow_not_converged and rc == 6):
+            self._check(rc)
+        return xs, [s.as_dict() for s in st]
+
+    def solve_multi_dev(self, xs, bs, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE,
+                        use_schur=True, allow_not_converged=False):
+        """Device-resident batched solve: lists of float64 CUDA tensors (full local slabs)."""
+        n = len(bs)
+        bp = (_P * n)(*[b.data_ptr() for b in bs])
+        xp = (_P * n)(*[x.data_ptr() for x in xs])
+        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur)
+        st = (SolveStats * n)()
+        rc = lib().qudax_solve_bicgstab_multi_dev(self._h, xp, bp, n, ctypes.byref(sp), st)
+        if rc and not (allow_not_converged and rc == 6):
+            self._check(rc)
+        return [s.as_dict() for s in st]
 
     def solve_dev(self, x, b, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
                   allow_not_converged=False, history=None):

@@ -44,3 +44,17 @@ def test_multi_rhs_bitwise_and_oracle(torch_cuda, prec, recon, nrhs):
         got = oracle.restrict(ctx.spinor_store(outs[k], prec, 0), 0)
         assert rel_l2(got, wc.matpc(oracle.restrict(psis[k], 0))) <= TOL[prec]
     ctx.close()
+
+
+def test_multirhs_fused_reductions_match_single(torch_cuda):
+    """Per-RHS fused reductions of the multi-RHS Mhat (through the batched solver's scalars):
+    covered bitwise by test_solver.test_batched_solve_equals_independent_solves; here the
+    error paths: the symmetric Schur form has no multi-RHS Mhat."""
+    import qgen
+    from paper_1011_0024_b200 import qudax
+    dims = (8, 4, 4, 8)
+    ctx = qudax.Context(dims)
+    ctx.gauge_load(qgen.gauge(dims, 7), 0.12, 1.0, prec=4, recon=12)
+    with pytest.raises(qudax.QudaxError):
+        ctx.solve_multi([qgen.point_source(dims, 0, 0)], use_schur=2)
+    ctx.close()

@@ -165,3 +165,45 @@ def test_symmetric_cgnr_vs_oracle(torch_cuda, system):
     assert res <= 1e-11
     assert abs(res - st["true_res"]) <= 1e-9
     ctx.close()
+
+
+@pytest.mark.parametrize("mode", [(4, 12, 0.1), (2, 12, 0.1)])
+def test_batched_solve_equals_independent_solves(torch_cuda, system, mode):
+    """Batched BiCGstab (6 sources per configuration): one
+    multi-RHS Mhat kernel pair per iteration with per-system fused reductions.  Every system's
+    iterations, reliable updates and solution are BITWISE those of its own single solve (same
+    per-site code, same per-CTA reduction slots), and the oracle confirms each true residual."""
+    U, wc = system
+    ps, rs, delta = mode
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=ps, recon_sloppy=rs, t_boundary=-1)
+    srcs = [qgen.point_source(DIMS, s, c) for s in (0, 1) for c in (0, 1, 2)]  # P:748-751
+    xs, sts = ctx.solve_multi(srcs, tol=1e-12, delta=delta, maxiter=5000, prec=8, prec_sloppy=ps)
+    for b, x, st in zip(srcs, xs, sts):
+        x1, st1 = ctx.solve(b, tol=1e-12, delta=delta, maxiter=5000, prec=8, prec_sloppy=ps)
+        assert (st["iters"], st["reliable_updates"]) == (st1["iters"], st1["reliable_updates"])
+        assert np.array_equal(x, x1)
+        res_oracle = np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b)
+        assert res_oracle <= 1e-12 * (1 + 1e-3) + 1e-15
+        assert abs(st["true_res"] - res_oracle) <= 1e-9
+    ctx.close()
+
+
+def test_batched_solve_mixed_convergence(torch_cuda, system):
+    """Systems that converge at different iterations leave the batch (the multi-RHS launches
+    shrink); a zero source converges at once; maxiter caps are reported per system."""
+    U, wc = system
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12, t_boundary=-1)
+    b0 = qgen.point_source(DIMS, 0, 0)
+    b1 = qgen.spinor(DIMS, 4242)          # a Gaussian source: more iterations than a point source
+    bz = np.zeros_like(b0)
+    xs, sts = ctx.solve_multi([b0, b1, bz], tol=1e-10, delta=0.1, maxiter=5000, prec=8, prec_sloppy=4)
+    assert sts[2]["iters"] == 0 and not np.any(xs[2])
+    assert sts[0]["iters"] != sts[1]["iters"]
+    for b, x in zip((b0, b1), xs[:2]):
+        assert np.linalg.norm(wc.M(x) - b) / np.linalg.norm(b) <= 1e-10 * (1 + 1e-3)
+    _, sts = ctx.solve_multi([b0, b1], tol=1e-14, delta=0.1, maxiter=7, prec=8, prec_sloppy=4,
+                             allow_not_converged=True)
+    assert all(s["iters"] == 7 for s in sts)
+    ctx.close()
