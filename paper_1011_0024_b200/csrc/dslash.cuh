@@ -711,18 +711,27 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // (multi-RHS launch: this CTA's right-hand side, recomputed here rather than kept live)
     const void *rh = a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat;
     SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx : rh, a.stride, i, w);
+#ifdef QX_RED_SITE_F64
+    using RA = double;
+#else
+    using RA = R;  // the site's 24-term partial in the arithmetic precision, sites summed in fp64
+#endif
+    RA s0 = 0, s1 = 0, s2 = 0;
 #pragma unroll
     for (int k = 0; k < 12; ++k) {
-        const double orr = o[2 * k], oi = o[2 * k + 1], wr = w[2 * k], wi = w[2 * k + 1];
+        const RA orr = o[2 * k], oi = o[2 * k + 1], wr = w[2 * k], wi = w[2 * k + 1];
         if (a.red_kind == RED_XDOT_NORM) {  // (<out, x>, |out|^2)
-            red[0] += orr * wr + oi * wi;
-            red[1] += orr * wi - oi * wr;
-            red[2] += orr * orr + oi * oi;
+            s0 += orr * wr + oi * wi;
+            s1 += orr * wi - oi * wr;
+            s2 += orr * orr + oi * oi;
         } else {                             // <rhat, out>
-            red[0] += wr * orr + wi * oi;
-            red[1] += wr * oi - wi * orr;
+            s0 += wr * orr + wi * oi;
+            s1 += wr * oi - wi * orr;
         }
     }
+    red[0] += (double)s0;
+    red[1] += (double)s1;
+    red[2] += (double)s2;
 }
 
 // Kernel-initiated halo (QUDAX_HALO_P2P): one thread per CTA acquires the two flags the
