@@ -34,7 +34,7 @@ sys.path.insert(0, ROOT)
 
 METRIC = "Dslash GFLOPS & HBM GB/s per B200 at 1/2/4/8 GPUs; mixed-prec solve time"
 KAPPA, CSW, EPS = 0.124, 1.0, 0.1
-SPATIAL, T_PER_GPU = 32, 64
+SPATIAL, T_PER_GPU, T_STRONG = 32, 64, 256
 GAUGE_SEED, SRC_SEED = 1005, 2005
 BLAS_FLOPS_PER_SITE_ITER = 960.0
 
@@ -51,6 +51,10 @@ def parse():
     ap.add_argument("--overlap", type=int, default=1)
     ap.add_argument("--halo", default="comm", choices=["comm", "p2p"],
                     help="N>1 spinor halo: NCCL send/recv (comm) or kernel-initiated over peer memory (p2p)")
+    ap.add_argument("--grid", default="", help="process grid Px,Py,Pz,Pt (default 1,1,1,N: T slabs, P:563-605; "
+                                               "others: multi-dimensional split, SURVEY 8(f) item 4)")
+    ap.add_argument("--scaling", default="weak", choices=["weak", "strong"],
+                    help="weak: 32^3x64 per GPU (BASELINE configs[4]); strong: 32^3x256 in total (configs[3])")
     return ap.parse_args()
 
 
@@ -280,8 +284,15 @@ def main():
     dev = torch.device("cuda", local)
     if world > 1:
         dist.init_process_group("nccl", device_id=dev)
-    dims = (SPATIAL, SPATIAL, SPATIAL, T_PER_GPU * N)
-    T_loc = T_PER_GPU
+    grid = tuple(int(v) for v in args.grid.split(",")) if args.grid else (1, 1, 1, N)
+    assert len(grid) == 4 and grid[0] * grid[1] * grid[2] * grid[3] == N, "grid must multiply to the GPU count"
+    if args.scaling == "weak":
+        local_dims = (SPATIAL, SPATIAL, SPATIAL, T_PER_GPU)
+        dims = tuple(l * p for l, p in zip(local_dims, grid))
+    else:
+        dims = (SPATIAL, SPATIAL, SPATIAL, T_STRONG)
+        local_dims = tuple(d // p for d, p in zip(dims, grid))
+    T_loc = local_dims[3]
 
     def barrier():
         if world > 1:
@@ -300,15 +311,16 @@ def main():
         obj = [qudax.nccl_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(obj, src=0)
         ctx = qudax.Context(dims, nranks=N, rank=rank, device=local, comm=qudax.COMM_NCCL, nccl_id=obj[0],
-                            overlap=bool(args.overlap),
+                            overlap=bool(args.overlap), proc_grid=grid,
                             halo=qudax.HALO_P2P if args.halo == "p2p" else qudax.HALO_COMM)
     else:
         ctx = qudax.Context(dims, device=local)
-    t0 = rank * T_loc
-    U = qgen.gauge(dims, GAUGE_SEED, eps=EPS, t_begin=t0, nt=T_loc)
+    assert ctx.local_dims == local_dims, (ctx.local_dims, local_dims)
+    origin = ctx.partition["origin"]
+    U = qgen.gauge_box(dims, GAUGE_SEED, origin, local_dims, eps=EPS)
     ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12, t_boundary=-1)
     del U
-    b_host = qgen.spinor(dims, SRC_SEED, t_begin=t0, nt=T_loc)
+    b_host = qgen.spinor_box(dims, SRC_SEED, origin, local_dims)
     with torch.cuda.stream(ctx.stream):
         b_dev = torch.from_numpy(b_host.view(np.float64)).to(dev)
         x_dev = torch.zeros_like(b_dev)
@@ -352,7 +364,7 @@ def main():
     achieved = ks["bytes_compulsory"] / (ks["ms_total"] * 1e-3) * 1e-9 if ks["ms_total"] > 0 else 0.0
     trafficd = profiled_traffic()
     traffic = None
-    if trafficd and trafficd.get("lattice") == [SPATIAL, SPATIAL, SPATIAL, T_loc]:
+    if trafficd and trafficd.get("lattice") == list(local_dims):
         traffic = trafficd.get("dram_bytes_per_launch")
     roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
                 "traffic": traffic, "kernel": "dslash_kernel fp32 recon-12 (clover-inverse + clover-xpay kinds)",
@@ -398,7 +410,7 @@ def main():
             k2 = ctx.kernel_stats(prec=prec)
             ctx.kernel_timing(False)
             m = qudax.site_model(prec, recon, -1)
-            sites = (SPATIAL ** 3 * T_loc // 2) * N
+            sites = (local_dims[0] * local_dims[1] * local_dims[2] * T_loc // 2) * N
             per_gpu = sites / N * reps
             dslash[name] = {
                 "matpc_gflops_total": m["flops"] * sites * reps / (mms * 1e-3) * 1e-9,
@@ -425,15 +437,19 @@ def main():
     if rank == 0:
         out = {
             "metric": METRIC, "value": value, "unit": "GFLOPS", "n_gpus": N, "steps": args.steps,
-            "warmup": args.warmup, "ms_per_step": ms / args.steps, "higher_is_better": True, "scaling": "weak",
+            "warmup": args.warmup, "ms_per_step": ms / args.steps, "higher_is_better": True, "scaling": args.scaling,
             "vs_baseline": None, "dtype": "f32", "data": "synthetic",
-            "config": {"workload": f"weak scaling 32^3x64 per GPU (global 32^3x{T_PER_GPU * N}), mixed-precision "
-                                   f"reliable-update BiCGstab, {args.iters} iterations per step (BASELINE configs[4])",
-                       "lattice_global": list(dims), "lattice_per_gpu": [SPATIAL, SPATIAL, SPATIAL, T_loc],
+            "config": {"workload": (f"weak scaling 32^3x64 per GPU (global {'x'.join(map(str, dims))}), "
+                                    if args.scaling == "weak" else
+                                    f"strong scaling 32^3x256 in total ({'x'.join(map(str, local_dims))} per GPU), ")
+                                   + f"mixed-precision reliable-update BiCGstab, {args.iters} iterations per step "
+                                   + ("(BASELINE configs[4])" if args.scaling == "weak" else "(BASELINE configs[3])"),
+                       "lattice_global": list(dims), "lattice_per_gpu": list(local_dims), "proc_grid": list(grid),
                        "precision": {"outer": "f64 recon-18", "sloppy": "f32 recon-12"},
                        "kappa": KAPPA, "csw": CSW, "gauge": f"weak field eps={EPS}", "t_boundary": "antiperiodic",
-                       "delta": 0.1, "parallelism": f"T-slab x{N}" + ((" (P2P kernel-initiated halo)" if args.halo == "p2p" else
-                                                         " (NCCL halo, overlapped)") if N > 1 else ""),
+                       "delta": 0.1, "parallelism": ("grid " + "x".join(map(str, grid)) if args.grid else f"T-slab x{N}")
+                                                    + ((" (P2P kernel-initiated halo)" if args.halo == "p2p" else
+                                                        " (NCCL halo, overlapped)") if N > 1 else ""),
                        "l2": "inputs larger than L2 (>1 GB of gauge+clover+fields per GPU vs 126 MB L2)"},
             "iters_per_step": iters / args.steps, "reliable_updates_per_step": updates / args.steps,
             "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches, "clocks": clocks,

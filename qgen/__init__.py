@@ -36,6 +36,8 @@ def _load():
         _lib.qgen_gauge.argtypes = [dp, ip, ctypes.c_int, ctypes.c_int, ctypes.c_uint64, ctypes.c_double]
         _lib.qgen_spinor.argtypes = [dp, ip, ctypes.c_int, ctypes.c_int, ctypes.c_uint64]
         _lib.qgen_gauge_transform.argtypes = [dp, ip, ctypes.c_int, ctypes.c_int, ctypes.c_uint64]
+        _lib.qgen_gauge_box.argtypes = [dp, ip, ip, ip, ctypes.c_uint64, ctypes.c_double]
+        _lib.qgen_spinor_box.argtypes = [dp, ip, ip, ip, ctypes.c_uint64]
     return _lib
 
 
@@ -64,6 +66,23 @@ def spinor(dims, seed, t_begin=0, nt=None):
     nt = T if nt is None else nt
     out = np.empty((nt, Z, Y, X, 4, 3), dtype=np.complex128)
     _load().qgen_spinor(_ptr(out), _dims(dims), int(t_begin), int(nt), int(seed))
+    return out
+
+
+def gauge_box(dims, seed, origin, extent, eps=-1.0):
+    """gauge() restricted to the box origin .. origin + extent (x, y, z, t order) of the global
+    lattice: [4, et, ez, ey, ex, 3, 3] — the same values as the corresponding slice of gauge()."""
+    ex, ey, ez, et = extent
+    out = np.empty((4, et, ez, ey, ex, 3, 3), dtype=np.complex128)
+    _load().qgen_gauge_box(_ptr(out), _dims(dims), _dims(origin), _dims(extent), int(seed), float(eps))
+    return out
+
+
+def spinor_box(dims, seed, origin, extent):
+    """spinor() restricted to a box: [et, ez, ey, ex, 4, 3]."""
+    ex, ey, ez, et = extent
+    out = np.empty((et, ez, ey, ex, 4, 3), dtype=np.complex128)
+    _load().qgen_spinor_box(_ptr(out), _dims(dims), _dims(origin), _dims(extent), int(seed))
     return out
 
 

@@ -167,3 +167,40 @@ void qgen_gauge_transform(double *out, const int dims[4], int t_begin, int nt, u
         memcpy(out + k * 18, m, sizeof(m));
     }
 }
+
+/* Sub-box generators (multi-dimensional partitioning): the same per-site counters as above on the
+ * box origin[mu] .. origin[mu] + ext[mu] - 1 of the global lattice (wrapped), so every rank of any
+ * process grid draws exactly its part of the one global field.
+ * gauge: double[4][et][ez][ey][ex][3][3][2]; spinor: double[et][ez][ey][ex][4][3][2]. */
+static inline uint64_t box_site(const int dims[4], const int o[4], long xl, long yl, long zl, long tl) {
+    const long X = dims[0], Y = dims[1], Z = dims[2], T = dims[3];
+    long xg = tmod(o[0] + xl, X), yg = tmod(o[1] + yl, Y), zg = tmod(o[2] + zl, Z), tg = tmod(o[3] + tl, T);
+    return (uint64_t)(((tg * Z + zg) * Y + yg) * X + xg);
+}
+void qgen_gauge_box(double *out, const int dims[4], const int o[4], const int e[4], uint64_t seed, double eps) {
+    const long V = (long)e[0] * e[1] * e[2] * e[3];
+#pragma omp parallel for schedule(static)
+    for (long k = 0; k < 4 * V; ++k) {
+        long mu = k / V, r = k % V;
+        long xl = r % e[0]; r /= e[0];
+        long yl = r % e[1]; r /= e[1];
+        long zl = r % e[2];
+        long tl = r / e[2];
+        double m[3][3][2];
+        su3_link(seed, box_site(dims, o, xl, yl, zl, tl), (uint32_t)mu, eps, m);
+        memcpy(out + k * 18, m, sizeof(m));
+    }
+}
+void qgen_spinor_box(double *out, const int dims[4], const int o[4], const int e[4], uint64_t seed) {
+    const long V = (long)e[0] * e[1] * e[2] * e[3];
+#pragma omp parallel for schedule(static)
+    for (long k = 0; k < V; ++k) {
+        long r = k;
+        long xl = r % e[0]; r /= e[0];
+        long yl = r % e[1]; r /= e[1];
+        long zl = r % e[2];
+        long tl = r / e[2];
+        const uint64_t site = box_site(dims, o, xl, yl, zl, tl);
+        for (uint32_t d = 0; d < 6; ++d) normals4(seed, 2u, site, 0u, d, out + k * 24 + 4 * d);
+    }
+}

@@ -58,6 +58,18 @@ def test_generator_su3_and_slab_independence():
     assert np.array_equal(qgen.spinor(dims, 5, t_begin=3, nt=2), psi[3:5])
 
 
+def test_generator_box_equals_global_slice():
+    """Process-grid boxes (multi-dimensional partitioning) draw exactly their part of the one
+    global field, wrapping at the lattice edge."""
+    dims = (8, 4, 6, 8)
+    U, S = qgen.gauge(dims, 5, eps=0.1), qgen.spinor(dims, 6)
+    ts, zs, ys, xs = [6, 7, 0, 1], [3, 4, 5], [0, 1, 2, 3], [4, 5, 6, 7]
+    g = qgen.gauge_box(dims, 5, (4, 0, 3, 6), (4, 4, 3, 4), eps=0.1)
+    s = qgen.spinor_box(dims, 6, (4, 0, 3, 6), (4, 4, 3, 4))
+    assert np.array_equal(g, U[:, ts][:, :, zs][:, :, :, ys][:, :, :, :, xs])
+    assert np.array_equal(s, S[ts][:, zs][:, :, ys][:, :, :, xs])
+
+
 def test_generator_haar_moments_and_weak_field():
     dims = (8, 8, 8, 8)
     U = qgen.gauge(dims, 3, eps=-1.0).reshape(-1, 3, 3)
