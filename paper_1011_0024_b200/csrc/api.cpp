@@ -260,6 +260,7 @@ static DslashArgs base_args(qudax_ctx *c, const qudax_ctx::GaugeCopy &gc, int pr
     const Geom &g = c->g;
     DslashArgs args{};
     args.X = g.X; args.Y = g.Y; args.Z = g.Z; args.T_loc = g.T_loc; args.Xh = g.Xh;
+    args.dXh = make_fastdiv(g.Xh); args.dY = make_fastdiv(g.Y); args.dZ = make_fastdiv(g.Z);
     args.Vh = (int)g.Vh; args.F = (int)g.F;
     args.stride = g.stride; args.fstride = g.fstride;
     args.parity = p;

@@ -586,6 +586,19 @@ struct RawVec {
             for (int r = 0; r < NREAL / 12; ++r) h[r].decode(scale, out + 12 * r);
         }
     }
+    // half: the stored integers plus the bias kHalfBias = 2^23 + 2^15, as fp32 (one PRMT per
+    // value, no arithmetic): the spatial projection removes the bias exactly (dslash.cuh)
+    __device__ __forceinline__ void decode_b(float *out) const {
+#pragma unroll
+        for (int r = 0; r < NREAL / 12; ++r) {
+            const uint32_t w[6] = {h[r].u.x, h[r].u.y, h[r].u.z, h[r].u.w, h[r].v.x, h[r].v.y};
+#pragma unroll
+            for (int k = 0; k < 6; ++k) {
+                out[12 * r + 2 * k] = __uint_as_float(__byte_perm(w[k], kHalfMagic, 0x7610));
+                out[12 * r + 2 * k + 1] = __uint_as_float(__byte_perm(w[k], kHalfMagic, 0x7632));
+            }
+        }
+    }
     // half: the stored integers; value = scale() * out
     __device__ __forceinline__ void decode_q(float *out) const {
 #pragma unroll

@@ -106,10 +106,35 @@ enum SiteRange { RANGE_ALL = 0, RANGE_INTERIOR = 1, RANGE_BOUNDARY = 2, RANGE_TA
 constexpr int kMaxRhs = 8;
 constexpr int kGroupHost = 64;  // = reduce.cuh kGroup (slots per tail group)
 
+// Division by a run-time constant d >= 1 for 0 <= n < 2^31 without the integer-division
+// emulation (I2F/MUFU/F2I + ~20 ALU/FMA instructions): q = umulhi(n, m) >> sh with
+// l = ceil(log2 d), m = floor(2^(31+l)/d) + 1, sh = l - 1 (Granlund-Montgomery; m*d - 2^(31+l)
+// is in (0, d] <= 2^l, so n*(m*d - 2^(31+l)) < 2^(31+l) and the quotient is exact).  d = 1:
+// m = 0 marks the identity.
+struct FastDiv {
+    unsigned m;
+    int sh, d;
+};
+inline FastDiv make_fastdiv(int d) {
+    FastDiv f{0u, 0, d};
+    if (d <= 1) return f;
+    int l = 0;
+    while ((1LL << l) < d) ++l;
+    f.m = (unsigned)(((1ULL << (31 + l)) / (unsigned long long)d) + 1ULL);
+    f.sh = l - 1;
+    return f;
+}
+#ifdef __CUDACC__
+__device__ __forceinline__ int fdiv(int n, const FastDiv &f) {
+    return f.m ? (int)(__umulhi((unsigned)n, f.m) >> f.sh) : n;
+}
+#endif
+
 struct DslashArgs {
     // geometry
     int X, Y, Z, T_loc, Xh;
     int Vh, F;
+    FastDiv dXh, dY, dZ;   // site index -> (xh, y, z, t) without integer division
     long stride, fstride;
     // partitioned X / Y / Z: bit mu of smask set -> hops off the local box
     // in mu read spin-projected half spinors (arithmetic precision) from sghost_{back,fwd}[mu]
