@@ -189,18 +189,18 @@ __device__ __forceinline__ float2 dq2_q(uint32_t w) {
                                  __uint_as_float(__byte_perm(w, kHalfMagic, 0x7632)));
     return __fadd2_rn(b, bc(-kHalfBias));
 }
-// two already-scaled floats -> packed offset-binary pair (round to nearest even)
-__device__ __forceinline__ uint32_t f32x2_to_i16x2(float a, float b) {
-    const uint32_t ia = __float_as_uint(__fadd_rn(a, 12615680.0f));  // 1.5*2^23 + 2^15
-    const uint32_t ib = __float_as_uint(__fadd_rn(b, 12615680.0f));
-    return __byte_perm(ia, ib, 0x5410);
+// a * inv, b * inv -> packed offset-binary pair: one FFMA2 rounds each exact product to the
+// nearest integer (even on ties) — one rounding, no intermediate fp32 product
+__device__ __forceinline__ uint32_t f32x2_scale_to_i16x2(float a, float b, float inv) {
+    const float2 r = __ffma2_rn(make_float2(a, b), bc(inv), bc(12615680.0f));  // 1.5*2^23 + 2^15
+    return __byte_perm(__float_as_uint(r.x), __float_as_uint(r.y), 0x5410);
+}
+// the integer round(x * inv) (exactly what f32x2_scale_to_i16x2 stores), as a float
+__device__ __forceinline__ float q_scaled_as_f32(float x, float inv) {
+    return __fmaf_rn(x, inv, 12582912.0f) - 12582912.0f;
 }
 // host/device: quantised integer q -> stored 16-bit word
 __host__ __device__ __forceinline__ short h16_code(int q) { return (short)(uint16_t)((unsigned)q ^ 0x8000u); }
-// the integer value held in a quantised word, as a float (exact)
-__device__ __forceinline__ float q_as_f32(float scaled) {
-    return __uint_as_float(__float_as_uint(__fadd_rn(scaled, 12582912.0f))) - 12582912.0f;
-}
 __device__ __forceinline__ uint2 ld_stream_u2(const uint2 *p) {
     uint2 v;
     asm volatile("ld.global.nc.L1::no_allocate.v2.u32 {%0,%1}, [%2];" : "=r"(v.x), "=r"(v.y) : "l"(p));
@@ -257,7 +257,7 @@ struct H12 {
     __device__ __forceinline__ void encode(const float *in, float inv) {
         uint32_t w[6];
 #pragma unroll
-        for (int k = 0; k < 6; ++k) w[k] = f32x2_to_i16x2(__fmul_rn(in[2 * k], inv), __fmul_rn(in[2 * k + 1], inv));
+        for (int k = 0; k < 6; ++k) w[k] = f32x2_scale_to_i16x2(in[2 * k], in[2 * k + 1], inv);
         u = make_uint4(w[0], w[1], w[2], w[3]);
         v = make_uint2(w[4], w[5]);
     }
@@ -337,7 +337,7 @@ struct SpinorIO {
             const float inv = (m > 0.f) ? kHalfMax / m : 0.f;
             const float scale = m * kHalfInv;
 #pragma unroll
-            for (int k = 0; k < 24; ++k) v[k] = __fmul_rn(scale, q_as_f32(__fmul_rn(v[k], inv)));
+            for (int k = 0; k < 24; ++k) v[k] = __fmul_rn(scale, q_scaled_as_f32(v[k], inv));
         }
     }
 };
