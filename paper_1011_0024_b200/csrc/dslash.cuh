@@ -22,6 +22,7 @@
 // L[15]; stored already halved): with u = spins 0,1 and l = spins 2,3 of the NR spinor,
 //   out_u = C+ (u + l) + C- (u - l),  out_l = C+ (u + l) - C- (u - l).
 #pragma once
+#include <cstdlib>
 #include "core.cuh"
 #include "internal.h"
 #include "reduce.cuh"
@@ -1056,10 +1057,23 @@ int dslash_blocks_prec(int recon, int dagger, int kind, int nthreads) {
     throw Error(QUDAX_ERR_ARG, "dslash: unsupported recon/kind");
 }
 
+#ifdef QX_MR_MINB
+template <int P, int NR> struct DslashMrMinBlocks { static constexpr int value = QX_MR_MINB; };
+#else
+template <int P, int NR> struct DslashMrMinBlocks { static constexpr int value = NR == 1 ? 6 : 4; };
+#endif
+}  // namespace qx
+#include "dslash_mr.cuh"
+namespace qx {
+
 template <int P, bool SS = false>
 void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
     const int threads = QX_DSLASH_THREADS;
     if (a.nthreads <= 0) return;
+    if constexpr (P != 8 && !SS) {  // several right-hand sides per thread (dslash_mr.cuh)
+        static const bool mr_off = std::getenv("QUDAX_MR_OFF") != nullptr;  // A/B: one RHS per thread
+        if (a.nrhs > 1 && !mr_off && launch_dslash_mr_prec<P>(recon, dagger, kind, a, s)) return;
+    }
 #define QX_DS(RC, DG, KD)                                                                       \
     if (recon == RC && dagger == DG && kind == KD) {                                            \
         dslash_kernel<P, RC, DG, KD, SS><<<dslash_blocks<P, RC, DG, KD>(a.nthreads) * (a.nrhs > 1 ? a.nrhs : 1), \
