@@ -8,8 +8,11 @@
 #include <algorithm>
 #include <chrono>
 #include <cmath>
+#include <cstdio>
 #include <cstdlib>
 #include <cstring>
+#include <map>
+#include <tuple>
 
 #include "ctx.h"
 
@@ -230,10 +233,20 @@ static void rec_model(const qudax_ctx::TimingRec &r, qudax_site_model *out) {
     out->bytes_paper = m.bytes_paper * r.sites * r.nrhs;
 }
 
+// QUDAX_TIMING_BREAKDOWN=1 (diagnostics): graph-replayed Dslash launch times per (precision,
+// kind, fused reduction), printed to stderr at finalize
+static std::map<std::tuple<int, int, int>, std::pair<long, double>> g_tbreak;
+static const bool g_tbreak_on = std::getenv("QUDAX_TIMING_BREAKDOWN") != nullptr;
+
 void harvest_graph_timing(qudax_ctx *c) {
     for (auto &r : c->graph_trecs) {
         float ms = 0;
         QX_CUDA(cudaEventElapsedTime(&ms, r.a, r.b));
+        if (g_tbreak_on) {
+            auto &e = g_tbreak[std::make_tuple(r.prec, r.kind, r.red)];
+            e.first += 1;
+            e.second += ms;
+        }
         qudax_site_model m;
         rec_model(r, &m);
         auto &t = c->tacc[prec_idx(r.prec)];
@@ -1162,6 +1175,10 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
 
 qudax_status qudax_finalize(qudax_ctx *c) {
     if (!c) return QUDAX_ERR_ARG;
+    if (g_tbreak_on)
+        for (auto &kv : g_tbreak)
+            std::fprintf(stderr, "qudax timing: prec %d kind %d red %d: %ld launches, %.2f us avg\n", std::get<0>(kv.first),
+                         std::get<1>(kv.first), std::get<2>(kv.first), kv.second.first, 1e3 * kv.second.second / kv.second.first);
     if (c->stream) cudaStreamSynchronize(c->stream);
     if (c->comm_stream) cudaStreamSynchronize(c->comm_stream);
     if (c->p2p.opened_fwd) cudaIpcCloseMemHandle(c->p2p.peer_fwd);
