@@ -484,6 +484,24 @@ __host__ __device__ constexpr bool dslash_hop_pf() {
     return (QX_HOP_PF >> (P == 2 ? 0 : (P == 4 ? 1 : 2))) & 1;
 }
 __device__ __forceinline__ void pf_l2(const void *p) { asm volatile("prefetch.global.L2 [%0];" ::"l"(p)); }
+__device__ __forceinline__ void pf_l1(const void *p) { asm volatile("prefetch.global.L1 [%0];" ::"l"(p)); }
+#ifndef QX_RED_PF
+#define QX_RED_PF 1
+#endif
+template <int P>
+__device__ __forceinline__ void pf_spinor_l1(const void *base, long stride, long j) {
+    if constexpr (P == 2) {
+        for (int h = 0; h < 2; ++h) {
+            pf_l1(cptr(base, h_spinor_u(stride, h) + 16 * j));
+            pf_l1(cptr(base, h_spinor_v(stride, h) + 8 * j));
+        }
+        pf_l1(cptr(base, (size_t)48 * stride + 4 * j));
+    } else {
+        constexpr int NB = (P == 8) ? 12 : 6;
+#pragma unroll
+        for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + j)));
+    }
+}
 // hf = -1: whole spinor, 0 / 1: upper / lower half
 template <int P>
 __device__ __forceinline__ void pf_spinor_l2(const void *base, long stride, long j, int hf) {
@@ -776,6 +794,15 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         };
         load_f();
         if constexpr (PAIR) load_b();
+#if QX_RED_PF
+        // the fused reduction's second operand (x or rhat0) is read right after the store: pull
+        // its lines into L1 while the last hops are computed (a dependent L2 round trip at the
+        // very end of every thread otherwise)
+        if (a.red_kind != RED_NONE) {
+            const void *w = a.red_kind == RED_XDOT_NORM ? fx : (a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat);
+            pf_spinor_l1<P>(w, a.stride, i);
+        }
+#endif
         if constexpr (dslash_hop_pf<P>() && !SS && (KIND == QUDAX_CLOVER_INV || KIND == QUDAX_CLOVER_INV_XPAY))
             pf_clover_l2<P>(a.clover, a.stride, i);
         {

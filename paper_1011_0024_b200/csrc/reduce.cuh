@@ -40,6 +40,18 @@ __device__ __forceinline__ void apply_coef(SolverScalars *S, int mode) {
     }
 }
 
+// Publishing a partial: a release atomic orders this thread's earlier slot stores before the
+// counter update (MEMBAR.ALL.GPU + ATOM) — __threadfence() + atomicAdd is a sequentially
+// consistent fence that also invalidates the SM's L1 (CCTL.IVALL) in every CTA, dropping the
+// neighbour spinors the other resident CTAs are reusing.  Only the CTA that finishes a group
+// acquires (and invalidates) before reading the other CTAs' slots.
+__device__ __forceinline__ unsigned atomic_add_release(unsigned *p, unsigned v) {
+    unsigned prev;
+    asm volatile("atom.add.release.gpu.global.u32 %0, [%1], %2;" : "=r"(prev) : "l"(p), "r"(v) : "memory");
+    return prev;
+}
+__device__ __forceinline__ void fence_acquire() { asm volatile("fence.acq_rel.gpu;" ::: "memory"); }
+
 // CTA-wide fixed-order sum of slots [b0, b1) of `src` (NRED values per slot) -> thread 0's out
 template <int NRED, int NT>
 __device__ __forceinline__ void cta_sum_slots(const double *src, int b0, int b1, double (&res)[NRED],
@@ -93,26 +105,24 @@ __device__ __forceinline__ void reduce_with_tail(double (&v)[NRED], const RedTai
             for (int w = 0; w < NT / 32; ++w) s += sm[w][k];
             t.partials[(size_t)gb * NRED + k] = s;
         }
-        __threadfence();
         const int gsize = min(kGroup, t.total_blocks - grp * kGroup);
-        const unsigned prev = atomicAdd(t.counter + 1 + grp, 1u);
+        const unsigned prev = atomic_add_release(t.counter + 1 + grp, 1u);
         stage = (prev == (unsigned)gsize - 1u) ? 1 : 0;
     }
     __syncthreads();
     if (stage == 0) return;
-    __threadfence();
+    fence_acquire();
     double res[NRED];
     cta_sum_slots<NRED, NT>(t.partials, grp * kGroup, min(t.total_blocks, (grp + 1) * kGroup), res, sm);
     if (threadIdx.x == 0) {
         for (int k = 0; k < NRED; ++k) gslots[(size_t)grp * NRED + k] = res[k];
         t.counter[1 + grp] = 0u;
-        __threadfence();
-        const unsigned prev = atomicAdd(t.counter, 1u);
+        const unsigned prev = atomic_add_release(t.counter, 1u);
         stage = (prev == (unsigned)ngroups - 1u) ? 2 : 0;
     }
     __syncthreads();
     if (stage != 2) return;
-    __threadfence();
+    fence_acquire();
     cta_sum_slots<NRED, NT>(gslots, 0, ngroups, res, sm);
     if (threadIdx.x == 0) {
         for (int k = 0; k < NRED; ++k) t.out[k] = res[k];
