@@ -1084,14 +1084,10 @@ int dslash_blocks_prec(int recon, int dagger, int kind, int nthreads) {
     throw Error(QUDAX_ERR_ARG, "dslash: unsupported recon/kind");
 }
 
-#ifdef QX_MR_MINB
-template <int P, int NR> struct DslashMrMinBlocks { static constexpr int value = QX_MR_MINB; };
-#else
-template <int P, int NR> struct DslashMrMinBlocks { static constexpr int value = NR == 1 ? 6 : 4; };
-#endif
-}  // namespace qx
-#include "dslash_mr.cuh"
-namespace qx {
+// several right-hand sides per thread (dslash_mr.cuh, instantiated in dslash_f{32,16}_mr.cu so
+// the two kernel families compile in parallel)
+bool launch_dslash_mr_f32(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
+bool launch_dslash_mr_f16(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
 
 template <int P, bool SS = false>
 void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
@@ -1099,7 +1095,9 @@ void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cu
     if (a.nthreads <= 0) return;
     if constexpr (P != 8 && !SS) {  // several right-hand sides per thread (dslash_mr.cuh)
         static const bool mr_off = std::getenv("QUDAX_MR_OFF") != nullptr;  // A/B: one RHS per thread
-        if (a.nrhs > 1 && !mr_off && launch_dslash_mr_prec<P>(recon, dagger, kind, a, s)) return;
+        if (a.nrhs > 1 && !mr_off &&
+            (P == 4 ? launch_dslash_mr_f32(recon, dagger, kind, a, s) : launch_dslash_mr_f16(recon, dagger, kind, a, s)))
+            return;
     }
 #define QX_DS(RC, DG, KD)                                                                       \
     if (recon == RC && dagger == DG && kind == KD) {                                            \

@@ -10,8 +10,15 @@
 // one.  Unpartitioned lattices only (RANGE_ALL, no ghosts); an odd last group repeats its
 // last RHS and skips its stores.
 #pragma once
+#include "dslash.cuh"
 
 namespace qx {
+
+#ifdef QX_MR_MINB
+template <int P, int NR> struct DslashMrMinBlocks { static constexpr int value = QX_MR_MINB; };
+#else
+template <int P, int NR> struct DslashMrMinBlocks { static constexpr int value = NR == 1 ? 6 : 4; };
+#endif
 
 #ifndef QX_MR_NR
 #define QX_MR_NR 2
