@@ -472,18 +472,7 @@ template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) 
 #else
 #define QX_MINB_OF(P) DslashMinBlocks<P>::value
 #endif
-// One-hop-ahead L2 prefetch (QX_HOP_PF bit mask per precision: 1 half, 2 fp32, 4 fp64): while a
-// direction's operands are in flight, prefetch.global.L2 of the next direction's neighbour
-// spinors and links (and, in the t direction, of the clover) — the next hop's DRAM latency
-// overlaps this hop's without holding registers.  A hint only.
-#ifndef QX_HOP_PF
-#define QX_HOP_PF 0
-#endif
-template <int P>
-__host__ __device__ constexpr bool dslash_hop_pf() {
-    return (QX_HOP_PF >> (P == 2 ? 0 : (P == 4 ? 1 : 2))) & 1;
-}
-__device__ __forceinline__ void pf_l2(const void *p) { asm volatile("prefetch.global.L2 [%0];" ::"l"(p)); }
+// L1 prefetch (QX_RED_PF: the fused reduction's second operand, see dslash_site)
 __device__ __forceinline__ void pf_l1(const void *p) { asm volatile("prefetch.global.L1 [%0];" ::"l"(p)); }
 #ifndef QX_RED_PF
 #define QX_RED_PF 1
@@ -502,57 +491,6 @@ __device__ __forceinline__ void pf_spinor_l1(const void *base, long stride, long
         for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + j)));
     }
 }
-// hf = -1: whole spinor, 0 / 1: upper / lower half
-template <int P>
-__device__ __forceinline__ void pf_spinor_l2(const void *base, long stride, long j, int hf) {
-    if constexpr (P == 2) {
-        for (int h = 0; h < 2; ++h) {
-            if (hf >= 0 && h != hf) continue;
-            pf_l2(cptr(base, h_spinor_u(stride, h) + 16 * j));
-            pf_l2(cptr(base, h_spinor_v(stride, h) + 8 * j));
-        }
-        pf_l2(cptr(base, (size_t)48 * stride + 4 * j));
-    } else {
-        constexpr int BPH = (P == 8) ? 6 : 3;
-#pragma unroll
-        for (int k = 0; k < 2 * BPH; ++k) {
-            if (hf >= 0 && k / BPH != hf) continue;
-            pf_l2(cptr(base, (size_t)16 * (k * stride + j)));
-        }
-    }
-}
-template <int P, int RECON>
-__device__ __forceinline__ void pf_link_l2(const void *base, long stride, long j) {
-    if constexpr (P == 2) {
-        constexpr int N16 = RECON / 8;
-        size_t off = 0;
-#pragma unroll
-        for (int k = 0; k < N16; ++k, off += (size_t)16 * stride) pf_l2(cptr(base, off + 16 * j));
-        if constexpr ((RECON % 8) >= 4) {
-            pf_l2(cptr(base, off + 8 * j));
-            off += (size_t)8 * stride;
-        }
-        if constexpr ((RECON % 4) == 2) pf_l2(cptr(base, off + 4 * j));
-    } else {
-        constexpr int NB = (P == 8) ? RECON / 2 : RECON / 4;
-#pragma unroll
-        for (int k = 0; k < NB; ++k) pf_l2(cptr(base, (size_t)16 * (k * stride + j)));
-        if constexpr (P == 4 && (RECON % 4) != 0) pf_l2(cptr(base, (size_t)16 * NB * stride + 8 * j));
-    }
-}
-template <int P>
-__device__ __forceinline__ void pf_clover_l2(const void *base, long stride, long j) {
-    if constexpr (P == 2) {
-#pragma unroll
-        for (int k = 0; k < 9; ++k) pf_l2(cptr(base, (size_t)16 * (k * stride + j)));
-        pf_l2(cptr(base, (size_t)144 * stride + 8 * j));
-    } else {
-        constexpr int NB = (P == 8) ? 36 : 18;
-#pragma unroll
-        for (int k = 0; k < NB; ++k) pf_l2(cptr(base, (size_t)16 * (k * stride + j)));
-    }
-}
-
 // one output site; red[] receives this site's contribution to the optional fused reduction
 // INMODE: load mode of the neighbour spinors (0 read-only path; 2 L2-coherent, for inputs
 // written by other CTAs earlier in the same launch — the fused Mhat kernel)
@@ -599,24 +537,6 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     constexpr int SF = DAG ? +1 : -1;  // sigma of the forward hop
     constexpr int SB = -SF;
 
-    // one-hop-ahead L2 prefetch of the next direction's operands (QX_HOP_PF A/B builds)
-    // (neighbour indices recomputed here so the default build keeps its register allocation)
-    auto hop_pf = [&](auto mu_c) {
-        constexpr int MU = decltype(mu_c)::value;
-        if constexpr (dslash_hop_pf<P>() && !SS) {
-            const int L = MU == 0 ? X : (MU == 1 ? Y : (MU == 2 ? Z : a.T_loc));
-            const int c = MU == 0 ? x : (MU == 1 ? y : (MU == 2 ? z : t));
-            const int st = MU == 0 ? 1 : (MU == 1 ? X : (MU == 2 ? XY : XYZ));
-            const int nf_ = (c == L - 1 ? lex - (L - 1) * st : lex + st) >> 1;
-            const int nb_ = (c == 0 ? lex + (L - 1) * st : lex - st) >> 1;
-            pf_spinor_l2<P>(fin, a.stride, nf_, MU == 3 ? (SF > 0 ? 0 : 1) : -1);
-            pf_spinor_l2<P>(fin, a.stride, nb_, MU == 3 ? (SB > 0 ? 0 : 1) : -1);
-            pf_link_l2<P, RECON>(a.gauge[MU][p], a.stride, i);
-            pf_link_l2<P, RECON>(a.gauge[MU][op], a.stride, nb_);
-        }
-    };
-
-    if (KIND == QUDAX_CLOVER_XPAY) hop_pf(std::integral_constant<int, 0>{});
     Cx<R> acc[4][3];
     // xpay: out = T x + a D in.  The site-local T x is computed FIRST and carried in the
     // accumulator as (1/a) T x, so its loads (x, clover) overlap the stencil's instead of
@@ -717,7 +637,6 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             sb.template load_spinor<INMODE>(bsrc, bstr, nb);
             lb.load(lbsrc, lbstr, lbi);
         }
-        if constexpr (MU < 3) hop_pf(std::integral_constant<int, MU + 1>{});
         if constexpr (DF && QX_BPROJ) {
             R v[24];
             Cx<R> ps[4][3], u[3][3], h0[3], h1[3];
@@ -803,8 +722,6 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             pf_spinor_l1<P>(w, a.stride, i);
         }
 #endif
-        if constexpr (dslash_hop_pf<P>() && !SS && (KIND == QUDAX_CLOVER_INV || KIND == QUDAX_CLOVER_INV_XPAY))
-            pf_clover_l2<P>(a.clover, a.stride, i);
         {
             R h[12];
             Cx<R> u[3][3];
@@ -919,116 +836,6 @@ __device__ __forceinline__ long p2p_wait(const DslashArgs &a) {
     return (s_seq & 1u) ? a.p2p_pdist : 0L;
 }
 
-// ---- CTA-level L2 prefetch of the streamed operands (TMA bulk prefetch).  The fp32 / half
-// kernels are memory-latency bound at their occupancy (6 x 128 threads per SM): one thread's
-// loads of a hop are only a few hundred bytes in flight.  Before any site is computed, warp 0
-// hands the copy engine one cp.async.bulk.prefetch.L2 per SoA region of every object the CTA
-// will stream (links of both hops, clover, x / rhat, the leading edge of the input spinor),
-// so the threads' demand loads meet lines already in (or on their way to) L2.  No registers
-// and no shared memory; a hint only (no effect on results).
-// Object layouts (bytes per site per region, in order): n16 16-byte regions, then n8 8-byte,
-// then n4 4-byte regions, each `stride` sites long (core.cuh).
-#ifndef QX_PREFETCH_MASK
-#define QX_PREFETCH_MASK 0
-#endif
-// bits: 1 forward links, 2 backward links, 4 clover, 8 x / rhat, 16 input-spinor leading edge
-#ifndef QX_PREFETCH_OBJS
-#define QX_PREFETCH_OBJS 31
-#endif
-template <int P>
-__host__ __device__ constexpr bool dslash_prefetch() {
-    return (QX_PREFETCH_MASK >> (P == 2 ? 0 : (P == 4 ? 1 : 2))) & 1;
-}
-struct PfObj {
-    unsigned char n16, n8, n4;
-};
-template <int P, int RECON>
-__device__ constexpr PfObj pf_link() {
-    if constexpr (P == 8) return {(unsigned char)(RECON / 2), 0, 0};
-    else if constexpr (P == 4) return {(unsigned char)(RECON / 4), (unsigned char)(RECON % 4 ? 1 : 0), 0};
-    else return {(unsigned char)(RECON / 8), (unsigned char)((RECON % 8) >= 4), (unsigned char)((RECON % 4) == 2)};
-}
-template <int P>
-__device__ constexpr PfObj pf_spinor() {
-    if constexpr (P == 8) return {12, 0, 0};
-    else if constexpr (P == 4) return {6, 0, 0};
-    else return {2, 2, 1};
-}
-template <int P>
-__device__ constexpr PfObj pf_clover() {
-    if constexpr (P == 8) return {36, 0, 0};
-    else if constexpr (P == 4) return {18, 0, 0};
-    else return {9, 1, 0};
-}
-__device__ __forceinline__ void l2_prefetch_bulk(const char *p, unsigned bytes) {
-    asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(p), "r"(bytes) : "memory");
-}
-// lane `lane` of the prefetching warp issues regions g = lane, lane + 32, ... of the object
-// sequence; returns the running region count.  [j0, j0 + n) sites, clamped into [0, Vh).
-__device__ __forceinline__ int pf_object(const void *base, PfObj o, long stride, long j0, int n, long Vh, int g0, int lane) {
-    if (base == nullptr) return g0;
-    if (j0 < 0) j0 = 0;
-    if (j0 + n > Vh) j0 = Vh - n;
-    if (j0 < 0) return g0;
-    const int nr = o.n16 + o.n8 + o.n4;
-    for (int r = (lane - g0 % 32 + 32) % 32; r < nr; r += 32) {
-        size_t off;
-        unsigned e;
-        if (r < o.n16) {
-            off = (size_t)16 * r * stride;
-            e = 16;
-        } else if (r < o.n16 + o.n8) {
-            off = (size_t)(16 * o.n16 + 8 * (r - o.n16)) * stride;
-            e = 8;
-        } else {
-            off = (size_t)(16 * o.n16 + 8 * o.n8 + 4 * (r - o.n16 - o.n8)) * stride;
-            e = 4;
-        }
-        const size_t b0 = (off + (size_t)e * j0) & ~(size_t)15;
-        const size_t b1 = (off + (size_t)e * (j0 + n) + 15) & ~(size_t)15;
-        l2_prefetch_bulk(static_cast<const char *>(base) + b0, (unsigned)(b1 - b0));
-    }
-    return g0 + nr;
-}
-template <int P, int RECON, int KIND>
-__device__ __forceinline__ void dslash_prefetch_cta(const DslashArgs &a, const void *fin, const void *fx, int blk, int rhs) {
-    if (threadIdx.x >= 32) return;
-    const int lane = threadIdx.x;
-    const int n = blockDim.x;
-    long t0 = (long)blk * n;
-    if (t0 >= a.nthreads) return;
-    long i0;
-    if (a.reverse) i0 = a.nthreads - t0 - n;  // sites [nthreads-1-t0-(n-1), nthreads-1-t0]
-    else i0 = t0;
-    if (a.range == RANGE_INTERIOR || a.range == RANGE_TAIL) i0 += a.F;
-    const long Vh = a.Vh;
-    const int p = a.parity, op = 1 - p;
-    constexpr int OB = QX_PREFETCH_OBJS;
-    int g = 0;
-    if (rhs == 0) {  // multi-RHS: the first CTA of a site block streams the shared operands
-        if (OB & 1)
-#pragma unroll
-            for (int mu = 0; mu < 4; ++mu) g = pf_object(a.gauge[mu][p], pf_link<P, RECON>(), a.stride, i0, n, Vh, g, lane);
-        if (OB & 2) {
-            const long sh[4] = {1, a.Xh, (long)a.X * a.Y / 2, (long)a.X * a.Y * a.Z / 2};
-#pragma unroll
-            for (int mu = 0; mu < 4; ++mu)
-                g = pf_object(a.gauge[mu][op], pf_link<P, RECON>(), a.stride, i0 - sh[mu], n, Vh, g, lane);
-        }
-        if ((OB & 4) && KIND != QUDAX_HOP) g = pf_object(a.clover, pf_clover<P>(), a.stride, i0, n, Vh, g, lane);
-    }
-    if (OB & 8) {
-        if (KIND == QUDAX_CLOVER_XPAY || KIND == QUDAX_CLOVER_INV_XPAY || a.red_kind == RED_XDOT_NORM)
-            g = pf_object(fx, pf_spinor<P>(), a.stride, i0, n, Vh, g, lane);
-        if (a.red_kind == RED_RHAT_DOT)
-            g = pf_object(a.nrhs > 1 ? a.rhat_m[rhs] : a.rhat, pf_spinor<P>(), a.stride, i0, n, Vh, g, lane);
-    }
-    if (OB & 16) {
-        const long lead = (long)a.X * a.Y * a.Z / 2;
-        g = pf_object(fin, pf_spinor<P>(), a.stride, a.reverse ? i0 - lead : i0 + lead, n, Vh, g, lane);
-    }
-}
-
 template <int P, int RECON, bool DAG, int KIND, bool SS>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
     // one thread per output site (a one-wave grid-stride variant measured 8-25% slower: the
@@ -1039,10 +846,6 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     if (a.nrhs > 1) {
         rhs = blk % a.nrhs;
         blk /= a.nrhs;
-    }
-    if constexpr (dslash_prefetch<P>() && !SS) {
-        if (a.range != RANGE_BOUNDARY) dslash_prefetch_cta<P, RECON, KIND>(a, a.nrhs > 1 ? a.in_m[rhs] : a.in,
-                                                                           a.nrhs > 1 ? a.x_m[rhs] : a.x, blk, rhs);
     }
     const int tid = blk * blockDim.x + threadIdx.x;
     double red[3] = {0.0, 0.0, 0.0};
