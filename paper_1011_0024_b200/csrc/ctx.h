@@ -112,6 +112,13 @@ struct qudax_ctx {
     double *dpart_m = nullptr;      // multi-RHS fused reductions: per-RHS CTA slots and counters
     unsigned *dcount_m = nullptr;
     double *stage = nullptr;  // fp64 full-slab staging (V_loc * 24 doubles)
+    // pageable host <-> device copies (api.cpp: h2d / d2h): a ring of pinned chunks that CPU
+    // threads fill (drain) while the copy engine moves the previous chunk
+    struct XferRing {
+        char *buf[4] = {};
+        cudaEvent_t done[4] = {};
+        size_t chunk = 0;
+    } xfer;
     int *d_flag = nullptr;
 
     // solver workspace (lazily allocated per (prec, prec_sloppy))
