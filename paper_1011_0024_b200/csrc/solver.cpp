@@ -296,12 +296,13 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
             convert_op(c, rs, Ps, r, Pd);
             rNorm = std::sqrt(r2);
             maxrr = rNorm;
-            if (updX || blown) {
+            const bool restart = blown;
+            if (updX || restart) {
                 r0Norm = rNorm;
                 maxrx = rNorm;
             }
             SolverScalars upd = hs;
-            if (blown) {  // restart: rhat0 = r, p = r (beta = 0, v = 0)
+            if (restart) {  // restart: rhat0 = r, p = r (beta = 0, v = 0)
                 copy(c, r0, rs, Ps);
                 zero(c, p, Ps);
                 zero(c, v, Ps);
@@ -497,9 +498,10 @@ void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_
                 convert_op(c, y.rs, Ps, y.r, Pd);
                 y.rNorm = std::sqrt(r2);
                 y.maxrr = y.rNorm;
-                if (updX || blown) y.r0Norm = y.maxrx = y.rNorm;
+                const bool restart = blown;
+                if (updX || restart) y.r0Norm = y.maxrx = y.rNorm;
                 SolverScalars upd = hs;
-                if (blown) {
+                if (restart) {
                     copy(c, y.r0, y.rs, Ps);
                     zero(c, y.p, Ps);
                     zero(c, y.v, Ps);

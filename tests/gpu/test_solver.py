@@ -207,3 +207,23 @@ def test_batched_solve_mixed_convergence(torch_cuda, system):
                              allow_not_converged=True)
     assert all(s["iters"] == 7 for s in sts)
     ctx.close()
+
+
+def test_half_sloppy_small_delta_stagnation_restart(torch_cuda):
+    """Double-half with a small reliable-update threshold (delta 3e-3) on a config-3 source
+    (24^3x128 weak field, colour 1 spin 0) whose residual decays by > 30 orders of magnitude
+    across the lattice: half-precision sites with norms below ~1e-34 made 32767/norm overflow,
+    the requantised values the fused reductions use turned into NaN (0 * inf), and every
+    iteration broke down and restarted (true residual stuck at 2.5e-3 after 4000 iterations,
+    scripts/diag_stall.py).  Such sites are now stored as zero (core.cuh kHalfTinyNorm)."""
+    import torch
+    dims = (24, 24, 24, 128)
+    U = qgen.gauge(dims, 1003, eps=0.1)
+    ctx = qudax.Context(dims)
+    ctx.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=2, recon_sloppy=12, t_boundary=-1)
+    b = torch.from_numpy(qgen.point_source(dims, 0, 1).view(np.float64).reshape(-1)).cuda()
+    x = torch.zeros_like(b)
+    st = ctx.solve_dev(x, b, tol=1e-14, delta=3e-3, maxiter=1500, prec=8, prec_sloppy=2, allow_not_converged=True)
+    assert st["true_res"] <= 1e-14 * (1 + 1e-3), st
+    assert st["iters"] < 600, st
+    ctx.close()
