@@ -12,6 +12,9 @@
 #include <cstdlib>
 #include <cstring>
 #include <map>
+#include <condition_variable>
+#include <functional>
+#include <mutex>
 #include <thread>
 #include <vector>
 #include <tuple>
@@ -74,27 +77,75 @@ static bool host_is_pinned(const void *p) {
     }
     return at.type == cudaMemoryTypeHost;
 }
-static void par_memcpy(void *dst, const void *src, size_t n) {
-    static const int nthr = [] {
+// A small persistent pool for the host copies (creating the threads per chunk cost more than
+// the copies' parallel speed-up).  Process-wide, started on first use, never torn down
+// (detached workers idle on a condition variable).
+class CopyPool {
+  public:
+    explicit CopyPool(int n) : n_(n) {
+        for (int t = 0; t < n_ - 1; ++t) std::thread([this, t] { worker(t + 1); }).detach();
+    }
+    int size() const { return n_; }
+    // run f(part) for part = 0 .. n-1 on the pool (part 0 on the caller), then return
+    template <typename F>
+    void run(F &&f) {
+        std::lock_guard<std::mutex> one_job(run_m_);  // contexts used from several host threads
+        std::unique_lock<std::mutex> lk(m_);
+        job_ = f;
+        pending_ = n_ - 1;
+        ++gen_;
+        lk.unlock();
+        cv_.notify_all();
+        f(0);
+        lk.lock();
+        done_.wait(lk, [&] { return pending_ == 0; });
+        job_ = nullptr;
+    }
+
+  private:
+    void worker(int id) {
+        unsigned seen = 0;
+        for (;;) {
+            std::function<void(int)> f;
+            {
+                std::unique_lock<std::mutex> lk(m_);
+                cv_.wait(lk, [&] { return gen_ != seen; });
+                seen = gen_;
+                f = job_;
+            }
+            f(id);
+            std::lock_guard<std::mutex> lk(m_);
+            if (--pending_ == 0) done_.notify_one();
+        }
+    }
+    int n_;
+    std::mutex run_m_, m_;
+    std::condition_variable cv_, done_;
+    std::function<void(int)> job_;
+    int pending_ = 0;
+    unsigned gen_ = 0;
+};
+static CopyPool &copy_pool() {
+    static CopyPool *pool = [] {
         const char *e = std::getenv("QUDAX_COPY_THREADS");
         const int hw = (int)std::thread::hardware_concurrency();
-        return e ? std::max(1, std::atoi(e)) : std::max(1, std::min(8, hw));
+        return new CopyPool(e ? std::max(1, std::atoi(e)) : std::max(1, std::min(8, hw)));
     }();
-    const size_t min_part = (size_t)2 << 20;
-    const int nt = (int)std::max<size_t>(1, std::min<size_t>(nthr, n / min_part));
-    if (nt == 1) {
+    return *pool;
+}
+static void par_memcpy(void *dst, const void *src, size_t n) {
+    auto &pool = copy_pool();
+    const int nt = pool.size();
+    if (nt == 1 || n < ((size_t)2 << 20)) {
         std::memcpy(dst, src, n);
         return;
     }
-    std::vector<std::thread> th;
     const size_t part = (n / nt + 63) & ~(size_t)63;
-    for (int t = 0; t < nt; ++t) {
+    pool.run([=](int t) {
         const size_t o = (size_t)t * part;
-        if (o >= n) break;
-        const size_t len = std::min(part, n - o);
-        th.emplace_back([=] { std::memcpy(static_cast<char *>(dst) + o, static_cast<const char *>(src) + o, len); });
-    }
-    for (auto &t : th) t.join();
+        if (o >= n) return;
+        std::memcpy(static_cast<char *>(dst) + o, static_cast<const char *>(src) + o, std::min(part, n - o));
+    });
 }
 static qudax_ctx::XferRing &xfer_ring(qudax_ctx *c) {
     auto &r = c->xfer;
