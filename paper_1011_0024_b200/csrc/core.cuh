@@ -480,7 +480,31 @@ struct LinkIO {
             for (int r = 0; r < 2; ++r)
 #pragma unroll
                 for (int c = 0; c < 3; ++c) u[r][c] = cx(raw[(r * 3 + c) * 2], raw[(r * 3 + c) * 2 + 1]);
-            // row2 = conj(row0 x row1)
+            // row2 = conj(row0 x row1).  Half precision (QX_XREC bit 0; bit 1 fp32, measured
+            // slower there): with conj(row 1) formed once, 4 FMUL2/FFMA2 per element (scalar
+            // broadcast / negation and the pair swap are operand modifiers) instead of two
+            // complex products, a subtraction and a conjugation (h-12 inverse-xpay -2 %)
+#ifndef QX_XREC
+#define QX_XREC 1
+#endif
+#if QX_XREC
+            if constexpr (sizeof(R) == 4 && (QX_XREC >> (P == 2 ? 0 : 1) & 1)) {
+                // conj(x y - z w) = x.r conj(y) - x.i swap(y) - z.r conj(w) + z.i swap(w)
+                float2 cy[3];
+#pragma unroll
+                for (int c = 0; c < 3; ++c) cy[c] = __fmul2_rn(f2(u[1][c]), make_float2(1.f, -1.f));
+                auto cross = [&](int xa, int yb, int za, int wb) {
+                    const Cx<float> xx = u[0][xa], zz = u[0][za];
+                    float2 r = __fmul2_rn(bc(xx.r), cy[yb]);
+                    r = __ffma2_rn(bc(-xx.i), make_float2(u[1][yb].i, u[1][yb].r), r);
+                    r = __ffma2_rn(bc(-zz.r), cy[wb], r);
+                    return cf(__ffma2_rn(bc(zz.i), make_float2(u[1][wb].i, u[1][wb].r), r));
+                };
+                const Cx<float> a0 = cross(1, 2, 2, 1), a1 = cross(2, 0, 0, 2), a2 = cross(0, 1, 1, 0);
+                u[2][0] = a0; u[2][1] = a1; u[2][2] = a2;
+                return;
+            }
+#endif
             u[2][0] = conj(u[0][1] * u[1][2] - u[0][2] * u[1][1]);
             u[2][1] = conj(u[0][2] * u[1][0] - u[0][0] * u[1][2]);
             u[2][2] = conj(u[0][0] * u[1][1] - u[0][1] * u[1][0]);
