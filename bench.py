@@ -58,7 +58,20 @@ def parse():
                                                "others: multi-dimensional split, SURVEY 8(f) item 4)")
     ap.add_argument("--scaling", default="weak", choices=["weak", "strong"],
                     help="weak: 32^3x64 per GPU (BASELINE configs[4]); strong: 32^3x256 in total (configs[3])")
+    ap.add_argument("--oracle-sample", type=int, default=0, help=argparse.SUPPRESS)  # internal: 1-thread oracle run
     return ap.parse_args()
+
+
+def cpu_oracle_1thread(iters=2):
+    """The same oracle sample on ONE host thread (oracle timed with nproc threads
+    and with 1), in a child process: OpenMP fixes its thread count at first use."""
+    import subprocess
+    env = dict(os.environ, OMP_NUM_THREADS="1")
+    r = subprocess.run([sys.executable, os.path.abspath(__file__), "--oracle-sample", str(iters)], env=env,
+                       capture_output=True, text=True, timeout=600)
+    if r.returncode != 0:
+        return None
+    return json.loads(r.stdout.strip().splitlines()[-1])
 
 
 # ---------------------------------------------------------------------------- clocks
@@ -269,6 +282,11 @@ def run_reference(args):
 
 # ---------------------------------------------------------------------------- our arm
 def main():
+    if "--oracle-sample" in sys.argv:  # child of cpu_oracle_1thread (no GPU work)
+        a = parse()
+        g, dt, threads, sample = cpu_oracle_gflops(a.oracle_sample)
+        print(json.dumps({"value": g, "seconds": dt, "cores": threads, "sample": sample}))
+        return
     args = parse()
     if args.impl == "reference":
         return run_reference(args)
@@ -435,6 +453,10 @@ def main():
     if rank == 0 and N == 1 and not args.no_cpu_baseline:
         g, dt, threads, sample = cpu_oracle_gflops(20)
         cpu = {"value": g, "unit": "GFLOPS", "cores": threads, "kind": "oracle", "sample": sample, "seconds": dt}
+        one = cpu_oracle_1thread(2)
+        if one:
+            cpu["one_thread"] = {"value": one["value"], "cores": one["cores"], "sample": one["sample"],
+                                 "seconds": one["seconds"]}
 
     ctx.close()
     if rank == 0:
