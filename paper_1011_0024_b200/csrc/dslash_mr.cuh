@@ -312,8 +312,12 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, DslashMrMinBlocks<P, NR>::v
     if (tid < a.nthreads) dslash_site_mr<P, RECON, DAG, KIND, NR>(a, tid, fin, fout, fx, frh, last_valid, red);
     if (a.red_kind != RED_NONE) {
 #pragma unroll
-        for (int r = 0; r < NR; ++r)
+        for (int r = 0; r < NR; ++r) {
+            // reduce_with_tail's shared scratch is reused by the next call: the CTA that finishes
+            // a reduction has thread 0 still reading it after the other threads return
+            if (r > 0) __syncthreads();
             if (r0 + r < a.nrhs) reduce_with_tail<3, QX_DSLASH_THREADS>(red[r], a.tail_m[r0 + r], blk);
+        }
     }
 }
 

@@ -227,3 +227,22 @@ def test_half_sloppy_small_delta_stagnation_restart(torch_cuda):
     assert st["true_res"] <= 1e-14 * (1 + 1e-3), st
     assert st["iters"] < 600, st
     ctx.close()
+
+
+def test_batched_equals_independent_at_config3_size(torch_cuda):
+    """Batched double-half solve of the six config-3 point sources (24^3x128) takes exactly the
+    iterations of the six independent solves.  Regression: the two-RHS-per-thread kernel ran
+    two fused reductions back to back, and the CTA finishing the first one still read the shared
+    scratch the second one was writing (rare, timing-dependent: a wrong global sum, then a
+    different Krylov sequence — iterations 150-163 instead of 141 for source 0)."""
+    dims = (24, 24, 24, 128)
+    U = qgen.gauge(dims, 1003, eps=0.1)
+    ctx = qudax.Context(dims)
+    ctx.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=2, recon_sloppy=12, t_boundary=-1)
+    srcs = [qgen.point_source(dims, s, c) for c in range(3) for s in range(2)]
+    _, sts = ctx.solve_multi(srcs, tol=1e-14, delta=1e-2, maxiter=1000, prec=8, prec_sloppy=2)
+    for b, st in zip(srcs, sts):
+        _, one = ctx.solve(b, tol=1e-14, delta=1e-2, maxiter=1000, prec=8, prec_sloppy=2)
+        assert (st["iters"], st["reliable_updates"]) == (one["iters"], one["reliable_updates"])
+        assert st["true_res"] <= 1e-14 * (1 + 1e-3)
+    ctx.close()
