@@ -83,6 +83,8 @@ __device__ __forceinline__ void cta_sum_slots(const double *src, int b0, int b1,
 // Layout: t.partials[0 .. total) CTA slots, then ceil(total/kGroup) group slots.
 // Counters: t.counter[0] groups done, t.counter[1 + g] CTAs done in group g (all zero on entry).
 // blk: this CTA's index within the reduction (-1: blockIdx.x)
+// Callers that run it twice in one kernel need a __syncthreads() between the calls: in the CTA
+// that finishes a reduction, thread 0 is still reading the shared scratch when the others return.
 template <int NRED, int NT>
 __device__ __forceinline__ void reduce_with_tail(double (&v)[NRED], const RedTail &t, int blk = -1) {
     __shared__ double sm[NT / 32][NRED];
