@@ -34,7 +34,9 @@
  *          qudax_spinor_bytes(ctx, prec) bytes, holding the V_h = V_loc/2 sites of one parity
  *          in the library's site-major SoA layout (eq. (4): N_int/N_vec blocks of
  *          V_h 16-byte short vectors; non-relativistic spin basis, eq. (6)).  Half precision
- *          appends one float norm per site.  The layout is opaque to callers:
+ *          appends one float norm per site (value = norm * q / 32767, norm = the
+ *          site's largest |component|; a site whose norm is <= 1e-30 is stored as zero,
+ *          DESIGN.md reading R6).  The layout is opaque to callers:
  *          move data in and out with qudax_spinor_load/store.  Reductions never see ghost
  *          zones: ghosts live in separate library-owned buffers.
  *
