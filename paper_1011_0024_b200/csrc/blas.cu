@@ -162,13 +162,59 @@ __global__ void k_tdot(long Vh, long stride, const void *t, const void *s, RedTa
 }
 
 // x <- x + alpha p + omega s ; s <- s - omega t ; returns (|s|^2, <rhat, s>) of the new s
+#ifndef QX_BICG_MINB
+#define QX_BICG_MINB 1
+#endif
 template <int P>
-__global__ void k_bicg_final(long Vh, long stride, void *x, const void *p, void *s, const void *t, const void *rhat,
+__global__ void __launch_bounds__(kBlasThreads, P == 4 ? QX_BICG_MINB : 1)
+k_bicg_final(long Vh, long stride, void *x, const void *p, void *s, const void *t, const void *rhat,
                              CoefArg alpha_, CoefArg omega_, RedTail tail) {
     using R = typename Prec<P>::R;
     const double2 alpha = coef_get(alpha_), omega = coef_get(omega_);
     const Cx<R> al = cx((R)alpha.x, (R)alpha.y), om = cx((R)omega.x, (R)omega.y);
     double acc[3] = {0, 0, 0};
+    if constexpr (P == 4) {
+        // fp32: one float4 block (two complex components) of all five fields at a time, in the
+        // site's component order (so every value and every fp64 partial sum is bitwise the
+        // whole-site version's): ~30 instead of 72 registers, 8 instead of 3 resident 256-thread
+        // CTAs per SM, and the loads of the next block in flight while this one is computed
+        // (the whole-site form was latency-bound at 0.78 of HBM, profiles/r01k_ncu_blas.txt)
+        QX_GRID_LOOP(i) {
+            float4 *X = reinterpret_cast<float4 *>(x);
+            float4 *Sv = reinterpret_cast<float4 *>(s);
+            const float4 *Pp = reinterpret_cast<const float4 *>(p), *T = reinterpret_cast<const float4 *>(t),
+                         *H = reinterpret_cast<const float4 *>(rhat);
+#pragma unroll
+            for (int k = 0; k < 6; ++k) {
+                const long j = (long)k * stride + i;
+                const float4 xv = __ldg(X + j), pv = __ldg(Pp + j), sv = __ldg(Sv + j), tv = __ldg(T + j), hv = __ldg(H + j);
+                const float xr[4] = {xv.x, xv.y, xv.z, xv.w}, pr[4] = {pv.x, pv.y, pv.z, pv.w};
+                const float sr[4] = {sv.x, sv.y, sv.z, sv.w}, tr[4] = {tv.x, tv.y, tv.z, tv.w};
+                const float hr[4] = {hv.x, hv.y, hv.z, hv.w};
+                float xo[4], so[4];
+#pragma unroll
+                for (int c = 0; c < 2; ++c) {
+                    const Cx<R> o = cx(xr[2 * c], xr[2 * c + 1]) + al * cx(pr[2 * c], pr[2 * c + 1]) +
+                                    om * cx(sr[2 * c], sr[2 * c + 1]);
+                    xo[2 * c] = o.r;
+                    xo[2 * c + 1] = o.i;
+                    const Cx<R> q = cx(sr[2 * c], sr[2 * c + 1]) - om * cx(tr[2 * c], tr[2 * c + 1]);
+                    so[2 * c] = q.r;
+                    so[2 * c + 1] = q.i;
+                }
+                X[j] = make_float4(xo[0], xo[1], xo[2], xo[3]);
+                Sv[j] = make_float4(so[0], so[1], so[2], so[3]);
+#pragma unroll
+                for (int c = 0; c < 2; ++c) {
+                    acc[0] += (double)so[2 * c] * so[2 * c] + (double)so[2 * c + 1] * so[2 * c + 1];
+                    acc[1] += (double)hr[2 * c] * so[2 * c] + (double)hr[2 * c + 1] * so[2 * c + 1];
+                    acc[2] += (double)hr[2 * c] * so[2 * c + 1] - (double)hr[2 * c + 1] * so[2 * c];
+                }
+            }
+        }
+        block_reduce_store<3>(acc, tail);
+        return;
+    }
     QX_GRID_LOOP(i) {
         R xx[24], pp[24], ss[24];
         SpinorIO<P>::load(x, stride, i, xx);
