@@ -66,7 +66,7 @@
 extern "C" {
 #endif
 
-#define QUDAX_ABI_VERSION 3
+#define QUDAX_ABI_VERSION 4
 
 typedef enum {
     QUDAX_OK = 0,
@@ -77,7 +77,8 @@ typedef enum {
     QUDAX_ERR_UNSUPPORTED = 5,   /* e.g. 8-reconstruct on near-singular links (reading Q6) */
     QUDAX_ERR_NOT_CONVERGED = 6, /* solver hit maxiter; x holds the last iterate */
     QUDAX_ERR_OOM = 7,           /* device allocation failed */
-    QUDAX_ERR_COMM = 8           /* host transport hook returned non-zero */
+    QUDAX_ERR_COMM = 8           /* host transport hook returned non-zero, or a kernel-initiated halo
+                                    wait timed out (a neighbour stalled: the result is not returned) */
 } qudax_status;
 
 typedef enum { QUDAX_HALF = 2, QUDAX_SINGLE = 4, QUDAX_DOUBLE = 8 } qudax_prec;
@@ -98,7 +99,9 @@ typedef enum { QUDAX_HOP = 0, QUDAX_CLOVER_INV = 1, QUDAX_CLOVER_XPAY = 2, QUDAX
  *   NONE  nranks must be 1; the Dslash wraps every dimension periodically inside one kernel.
  *   NCCL  ncclSend/ncclRecv of spin-projected faces on a comm stream, overlapped with the
  *         interior kernel; ncclAllReduce for global sums.  With
- *         nranks == 1 this is the loopback test mode (faces go through NCCL to self).
+ *         nranks == 1 this is the loopback test mode: faces go through NCCL to self and every
+ *         global sum through ncclAllReduce on the one-rank communicator, so the N > 1 code
+ *         path (including its CUDA-graph capture) runs on one GPU.
  *   Faces: T faces carry the 12 reals the diagonal temporal projector keeps, in the storage
  *         precision (bits only, half with its norm; eq. (6)).  Faces of a partitioned
  *         X, Y or Z carry the spin-projected half spinor (1 -+ gamma_mu) psi (footnote 3,
@@ -126,6 +129,16 @@ typedef enum { QUDAX_COMM_NONE = 0, QUDAX_COMM_NCCL = 1, QUDAX_COMM_HOST = 2 } q
  *         neighbour is the rank itself: the loopback test of the kernel path.  P2P supports a
  *         T-only split (split_mask = T); other grids return QUDAX_ERR_UNSUPPORTED at init. */
 typedef enum { QUDAX_HALO_COMM = 0, QUDAX_HALO_P2P = 1 } qudax_halo_kind;
+
+/* Behaviour flags of qudax_init_param.flags (0 = the defaults every measurement uses).  Test and
+ * comparison switches only; none changes a result beyond its documented rounding. */
+typedef enum {
+    QUDAX_FLAG_NO_GRAPHS = 1,          /* solver iterations enqueued eagerly, not replayed as CUDA graphs */
+    QUDAX_FLAG_DEBUG_SOLVER = 2,       /* per-iteration solver scalars to stderr */
+    QUDAX_FLAG_FORCE_SS = 4,           /* the partitioned-X/Y/Z kernel instantiation on every lattice (test) */
+    QUDAX_FLAG_ONE_RHS_PER_THREAD = 8, /* multi-RHS launches with one right-hand side per thread (comparison) */
+    QUDAX_FLAG_TIMING_BREAKDOWN = 16   /* per-(precision, kind, reduction) Dslash times to stderr at finalize */
+} qudax_init_flag;
 
 typedef struct qudax_ctx qudax_ctx;
 
@@ -163,6 +176,9 @@ typedef struct {
                                     nranks == 1 with a transport (loopback).  A non-zero mask must
                                     contain every dimension with P_mu > 1; extra bits are loopback
                                     dimensions (the rank is its own neighbour) for tests. */
+    int flags;                   /* qudax_init_flag bits (0 = defaults) */
+    int copy_threads;            /* host threads of the pageable host<->device copies (0 = min(8, cores));
+                                    process-wide, fixed by the first context that copies */
 } qudax_init_param;
 
 typedef struct {
@@ -184,6 +200,11 @@ typedef struct {
     double *res_history;         /* optional host array: ||r_k|| / ||bhat|| after iteration k (the
                                     iterated residual, replaced by the true one at reliable updates) */
     int history_cap;             /* capacity of res_history (0 = none) */
+    int poll_every;              /* BiCGstab: iterations enqueued (one CUDA graph) between host reads of
+                                    the device-side scalars, 1..64 (0 = 4).  Algorithm R's update rule is
+                                    evaluated on the device after every iteration; an iteration that
+                                    calls for a reliable update stops the rest of the batch (its kernels
+                                    return at once), so the iterates do not depend on poll_every. */
 } qudax_solve_param;
 
 typedef struct {

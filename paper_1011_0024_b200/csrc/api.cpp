@@ -125,11 +125,11 @@ class CopyPool {
     int pending_ = 0;
     unsigned gen_ = 0;
 };
+static int g_copy_threads = 0;  // qudax_init_param.copy_threads of the first context (0 = default)
 static CopyPool &copy_pool() {
     static CopyPool *pool = [] {
-        const char *e = std::getenv("QUDAX_COPY_THREADS");
         const int hw = (int)std::thread::hardware_concurrency();
-        return new CopyPool(e ? std::max(1, std::atoi(e)) : std::max(1, std::min(8, hw)));
+        return new CopyPool(g_copy_threads > 0 ? g_copy_threads : std::max(1, std::min(8, hw)));
     }();
     return *pool;
 }
@@ -196,7 +196,7 @@ static void d2h(qudax_ctx *c, void *dst, const void *src, size_t n) {
     }
 }
 
-static void dfree(qudax_ctx *c, void *p) {
+void dfree(qudax_ctx *c, void *p) {
     if (!p) return;
     auto it = std::find(c->allocs.begin(), c->allocs.end(), p);
     if (it != c->allocs.end()) c->allocs.erase(it);
@@ -310,6 +310,9 @@ static void exchange(qudax_ctx *c, const void *send_fwd, const void *send_back, 
 }
 
 static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res);
+// whether a reduction's local sums must go through the transport before they are used: several
+// ranks, or the NCCL loopback at one rank (which runs the N > 1 code path on one GPU)
+static bool global_sums(const qudax_ctx *c) { return c->g.nranks > 1 || c->comm == QUDAX_COMM_NCCL; }
 
 static cudaEvent_t pool_event(qudax_ctx *c) {
     if (!c->ev_pool.empty()) {
@@ -343,7 +346,7 @@ static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int
         return;
     }
     qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads, a.nrhs > 1 ? a.nrhs : 1,
-                           a.red_kind};
+                           a.red_kind, c->cap_iter};
     if (c->capturing) {  // graph: external event-record nodes, re-recorded at each replay
         QX_CUDA(cudaEventRecordWithFlags(r.a, c->stream, cudaEventRecordExternal));
         launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
@@ -372,16 +375,18 @@ static void rec_model(const qudax_ctx::TimingRec &r, qudax_site_model *out) {
     out->bytes_paper = m.bytes_paper * r.sites * r.nrhs;
 }
 
-// QUDAX_TIMING_BREAKDOWN=1 (diagnostics): graph-replayed Dslash launch times per (precision,
+// QUDAX_FLAG_TIMING_BREAKDOWN (diagnostics): graph-replayed Dslash launch times per (precision,
 // kind, fused reduction), printed to stderr at finalize
 static std::map<std::tuple<int, int, int>, std::pair<long, double>> g_tbreak;
-static const bool g_tbreak_on = std::getenv("QUDAX_TIMING_BREAKDOWN") != nullptr;
 
-void harvest_graph_timing(qudax_ctx *c) {
-    for (auto &r : c->graph_trecs) {
+// the timing records of one replay of a captured graph (only those of the first `iters` solver
+// iterations of the batch: the later ones were halted and ran no work)
+void harvest_graph_timing(qudax_ctx *c, const std::vector<qudax_ctx::TimingRec> &recs, int iters) {
+    for (auto &r : recs) {
+        if (r.iter >= iters) continue;
         float ms = 0;
         QX_CUDA(cudaEventElapsedTime(&ms, r.a, r.b));
-        if (g_tbreak_on) {
+        if (c->flags & QUDAX_FLAG_TIMING_BREAKDOWN) {
             auto &e = g_tbreak[std::make_tuple(r.prec, r.kind, r.red)];
             e.first += 1;
             e.second += ms;
@@ -398,12 +403,20 @@ void harvest_graph_timing(qudax_ctx *c) {
     }
 }
 
-void release_graph_timing(qudax_ctx *c) {
-    for (auto &r : c->graph_trecs) {
+void check_device_error(qudax_ctx *c) {
+    if (c->h_err && *reinterpret_cast<volatile int *>(c->h_err)) {
+        *reinterpret_cast<volatile int *>(c->h_err) = 0;
+        throw Error(QUDAX_ERR_COMM, "kernel-initiated halo: a neighbour's face flag did not arrive (wait timed out); "
+                                    "the operator result is invalid");
+    }
+}
+
+void release_graph_timing(qudax_ctx *c, std::vector<qudax_ctx::TimingRec> &recs) {
+    for (auto &r : recs) {
         c->ev_pool.push_back(r.a);
         c->ev_pool.push_back(r.b);
     }
-    c->graph_trecs.clear();
+    recs.clear();
 }
 
 // kernel arguments common to every Dslash launch of (precision, output parity, kind)
@@ -421,6 +434,10 @@ static DslashArgs base_args(qudax_ctx *c, const qudax_ctx::GaugeCopy &gc, int pr
     args.bc_back = (g.c[3] == 0) ? (double)c->t_bc : 1.0;
     args.a = a;
     args.reverse = reverse;
+    args.halt = c->halt;
+    args.err = c->d_err;
+    args.variant = ((c->flags & QUDAX_FLAG_FORCE_SS) ? kVariantForceSS : 0) |
+                   ((c->flags & QUDAX_FLAG_ONE_RHS_PER_THREAD) ? kVariantOneRhsPerThread : 0);
     args.nrhs = 1;
     for (int m = 0; m < 4; ++m)
         for (int q = 0; q < 2; ++q) args.gauge[m][q] = gc.d[m][q];
@@ -457,7 +474,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
     const long n_int = g.n_int, n_bnd = g.Vh - g.n_int;
     const bool split = c->comm == QUDAX_COMM_NCCL && !c->p2p.on && c->overlap && n_int > 0;
-    const bool multi = (g.nranks > 1);  // cross-rank sums needed before the scalar recurrence
+    const bool multi = global_sums(c);  // sums go through the transport before the recurrence
     if (red) {
         QX_CHECK(red->kind != RED_XDOT_NORM || kind >= QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
         QX_CHECK(red->kind != RED_RHAT_DOT || red->rhat, QUDAX_ERR_ARG, "rhat-dot needs rhat");
@@ -503,7 +520,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
                                   q.pdist[pi], reinterpret_cast<unsigned *>(q.peer_back + q.off_flags) + 1,
                                   reinterpret_cast<unsigned *>(q.peer_fwd + q.off_flags),
                                   reinterpret_cast<unsigned *>(q.base + q.off_seq),
-                                  reinterpret_cast<unsigned *>(q.base + q.off_count), st);
+                                  reinterpret_cast<unsigned *>(q.base + q.off_count), c->halt, st);
             c->launches += 1;
         };
         if (c->overlap && g.T_loc > 2) {
@@ -547,11 +564,11 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     if (g.split & 8) xf[nx++] = Xfer{3, h.sf, h.sb, h.gb, h.gf, h.bytes, h.h_sf, h.h_sb, h.h_gb, h.h_gf};
     auto pack_all = [&](cudaStream_t st) {
         if (g.split & 8) {
-            launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, st);
+            launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, c->halt, st);
             c->launches += 1;
         }
         if (spatial_split(g)) {
-            launch_pack_spatial(prec, dagger, g, 1 - p, in, h.ssb, h.ssf, st);
+            launch_pack_spatial(prec, dagger, g, 1 - p, in, h.ssb, h.ssf, c->halt, st);
             c->launches += 1;
         }
     };
@@ -590,85 +607,6 @@ static void *tmp_even(qudax_ctx *c, int prec) {
 }
 
 // Mhat = T_ee - kappa^2 D_eo T_oo^{-1} D_oe (asymmetric Schur form on even sites)
-// dispense order of the fused Mhat wavefront (matpc_fused.cuh): A(0..L), then A(k) followed
-// by B(k-L), then the remaining B's; B(0) last (it needs A(T-1) through the periodic wrap).
-static const int *fused_stages(qudax_ctx *c) {
-    if (c->fstages) return c->fstages;
-    const int T = c->g.T_loc;
-    const char *lag = std::getenv("QUDAX_FUSED_LAG");
-    const int L = lag ? std::max(1, std::atoi(lag)) : 1;
-    std::vector<int> st;
-    for (int k = 0; k <= std::min(L, T - 1); ++k) st.push_back(k);
-    std::vector<bool> bdone(T, false);
-    for (int k = L + 1; k < T; ++k) {
-        st.push_back(k);
-        const int b = k - L;
-        if (b >= 1) { st.push_back(T + b); bdone[b] = true; }
-    }
-    for (int b = 1; b < T; ++b)
-        if (!bdone[b]) st.push_back(T + b);
-    st.push_back(T + 0);
-    QX_CHECK((int)st.size() == 2 * T, QUDAX_ERR_STATE, "fused stage table");
-    int *d = static_cast<int *>(dalloc(c, sizeof(int) * st.size()));
-    QX_CUDA(cudaMemcpy(d, st.data(), sizeof(int) * st.size(), cudaMemcpyHostToDevice));
-    c->fcounters = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * (T + 1)));
-    c->fstages = d;
-    return d;
-}
-
-// Mhat as one persistent wavefront launch (unpartitioned contexts)
-static void matpc_fused(qudax_ctx *c, void *out, const void *in, void *t, int prec, int dagger, const RedReq *red) {
-    auto &gc = gauge_for(c, prec);
-    const Geom &g = c->g;
-    const int TPB = dslash_threads();
-    FusedArgs f{};
-    f.A = base_args(c, gc, prec, 1, QUDAX_CLOVER_INV, 0.0, 0);
-    f.A.in = in; f.A.out = t; f.A.ghosted = 0; f.A.range = RANGE_ALL; f.A.nthreads = (int)g.Vh;
-    f.B = base_args(c, gc, prec, 0, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, 0);
-    f.B.in = t; f.B.x = in; f.B.out = out; f.B.ghosted = 0; f.B.range = RANGE_ALL; f.B.nthreads = (int)g.Vh;
-    f.chunks = (int)((g.F + TPB - 1) / TPB);
-    f.total_items = 2 * g.T_loc * f.chunks;
-    f.stages = fused_stages(c);
-    f.work = c->fcounters;
-    f.doneA = c->fcounters + 1;
-    const int wave = prec == 8 ? matpc_fused_wave_f64(gc.recon, dagger)
-                               : (prec == 4 ? matpc_fused_wave_f32(gc.recon, dagger) : matpc_fused_wave_f16(gc.recon, dagger));
-    const int grid = std::min(wave, f.total_items);
-    if (red) {
-        QX_CHECK(red->kind == RED_RHAT_DOT ? red->rhat != nullptr : red->kind == RED_XDOT_NORM, QUDAX_ERR_ARG,
-                 "fused matpc: bad reduction");
-        if (!c->dpart) c->dpart = static_cast<double *>(dalloc(c, sizeof(double) * 3 * (2 * (g.Vh / 32) + 64)));
-        f.B.red_kind = red->kind;
-        f.B.rhat = red->rhat;
-        f.B.tail.partials = c->dpart;
-        f.B.tail.counter = c->d_counter;
-        f.B.tail.total_blocks = grid;
-        f.B.tail.block_offset = 0;
-        f.B.tail.out = red->S ? red->S->red : c->red_out;
-        f.B.tail.S = red->S;
-        f.B.tail.coef_mode = red->S ? red->coef_mode : COEF_NONE;
-    }
-    QX_CUDA(cudaMemsetAsync(c->fcounters, 0, sizeof(unsigned) * (g.T_loc + 1), c->stream));
-    auto launch = [&] {
-        if (prec == 8) launch_matpc_fused_f64(gc.recon, dagger, f, grid, c->stream);
-        else if (prec == 4) launch_matpc_fused_f32(gc.recon, dagger, f, grid, c->stream);
-        else launch_matpc_fused_f16(gc.recon, dagger, f, grid, c->stream);
-        QX_CUDA(cudaGetLastError());
-    };
-    if (c->timing) {
-        qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, gc.recon, -2, (long)g.Vh, 1};
-        const unsigned fl = c->capturing ? cudaEventRecordExternal : cudaEventRecordDefault;
-        QX_CUDA(cudaEventRecordWithFlags(r.a, c->stream, fl));
-        launch();
-        QX_CUDA(cudaEventRecordWithFlags(r.b, c->stream, fl));
-        (c->capturing ? c->graph_trecs : c->trecs).push_back(r);
-    } else {
-        launch();
-    }
-    c->launches += 1;
-    if (red && !red->S) global_sum(c, c->red_out, 3, red->res);
-}
-
 // symmetric Schur form: T_ee^{-1} Mhat.  Non-dagger: CLOVER_INV on odd,
 // CLOVER_INV_XPAY on even (fused reductions as for Mhat).  Dagger (explicit adjoint, not
 // gamma5-Hermitian): T_ee^{-1} in -> CLOVER_INV^dag on odd -> HOP^dag on even -> in - kappa^2 (.)
@@ -698,10 +636,6 @@ void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, con
         return;
     }
     void *t = tmp_odd(c, prec);
-    if (c->comm == QUDAX_COMM_NONE && c->fused && c->g.T_loc >= 2) {
-        matpc_fused(c, out, in, t, prec, dagger, red);
-        return;
-    }
     dslash_op(c, t, in, nullptr, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, nullptr);
     // the second kernel walks the lattice top-down: the timeslices the first kernel touched
     // last (their links, T^{-1} D in and the dirty tmp lines) are still in the 126 MB L2
@@ -784,7 +718,7 @@ void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int pari
 }
 
 static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res) {
-    if (c->g.nranks > 1 && c->comm == QUDAX_COMM_NCCL) {
+    if (c->comm == QUDAX_COMM_NCCL) {  // (one rank: the loopback test of the N > 1 path)
         QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl, c->stream));
     }
     QX_CUDA(cudaMemcpyAsync(c->h_red, dev_vals, sizeof(double) * n, cudaMemcpyDeviceToHost, c->stream));
@@ -802,7 +736,7 @@ int blas_op(qudax_ctx *c, int op, int prec, void *const *f, const double *coef, 
         if (op == OP_P_UPDATE || op == OP_FINAL) co[1].v = make_double2(coef[2], coef[3]);
     }
     RedTail tail{c->partials, c->d_counter, 0, 0, c->red_out, nullptr, COEF_NONE};
-    int n = blas_run(op, prec, c->g, f, co, tail, c->stream);
+    int n = blas_run(op, prec, c->g, f, co, tail, c->halt, c->stream);
     c->launches += 1;
     if (n) global_sum(c, c->red_out, n, res);
     return n;
@@ -811,7 +745,7 @@ int blas_op(qudax_ctx *c, int op, int prec, void *const *f, const double *coef, 
 // Global sum of n device doubles in place (stream-ordered, no host round trip for NCCL / one
 // rank), then the device-side scalar recurrence `mode` (launch_coef).
 void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, int mode) {
-    if (c->g.nranks > 1 && c->comm == QUDAX_COMM_NCCL) {
+    if (c->comm == QUDAX_COMM_NCCL) {  // (one rank: the loopback test of the N > 1 path)
         QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl, c->stream));
     } else if (c->g.nranks > 1 && c->comm == QUDAX_COMM_HOST) {
         QX_CUDA(cudaMemcpyAsync(c->h_red, dev_vals, sizeof(double) * n, cudaMemcpyDeviceToHost, c->stream));
@@ -820,7 +754,7 @@ void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, in
         QX_CUDA(cudaMemcpyAsync(dev_vals, c->h_red, sizeof(double) * n, cudaMemcpyHostToDevice, c->stream));
     }
     if (mode != COEF_NONE) {
-        launch_coef(S, mode, c->stream);
+        launch_coef(S, mode, c->halt, c->stream);
         c->launches += 1;
     }
 }
@@ -828,9 +762,9 @@ void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, in
 // BLAS op whose coefficients may live on the device; its reduction (if any) goes to S->red,
 // is summed over ranks and fed to the scalar recurrence `mode` — all stream-ordered.
 void blas_op_dev(qudax_ctx *c, int op, int prec, void *const *f, const CoefArg *co, SolverScalars *S, int mode) {
-    const bool multi = c->g.nranks > 1;
+    const bool multi = global_sums(c);
     RedTail tail{c->partials, c->d_counter, 0, 0, S->red, S, multi ? COEF_NONE : mode};
-    int n = blas_run(op, prec, c->g, f, co, tail, c->stream);
+    int n = blas_run(op, prec, c->g, f, co, tail, c->halt, c->stream);
     c->launches += 1;
     if (n && multi) device_sum_coef(c, S->red, n, S, mode);
 }
@@ -870,6 +804,8 @@ static void gauge_load(qudax_ctx *c, const double *host, const qudax_gauge_param
     }
     c->ncopies = 0;
     c->gauge_loaded = false;
+    c->gauge_epoch += 1;  // cached solver graphs baked in the old gauge / clover pointers
+    drop_graphs(c);
     c->kappa = p->kappa;
     c->csw = p->csw;
     c->t_bc = p->t_boundary;
@@ -1161,22 +1097,44 @@ static void setup_p2p(qudax_ctx *c) {
         return;
     }
     static_assert(sizeof(cudaIpcMemHandle_t) == 64, "IPC handle size");
-    cudaIpcMemHandle_t mine, hb, hf;
-    QX_CUDA(cudaIpcGetMemHandle(&mine, q.base));
+    // each rank sends {IPC handle, PCI bus id of its GPU}: a neighbour on another GPU must be
+    // reachable by peer access (NVLink / NVSwitch on a B200 node), else UNSUPPORTED — the comm
+    // halo (NCCL) is the path for GPUs without peer access
+    struct Rec {
+        cudaIpcMemHandle_t h;
+        char bus[64];
+    };
+    Rec mine{}, rb{}, rf{};
+    QX_CUDA(cudaIpcGetMemHandle(&mine.h, q.base));
+    QX_CUDA(cudaDeviceGetPCIBusId(mine.bus, sizeof(mine.bus), c->device));
     if (c->comm == QUDAX_COMM_HOST) {
-        cudaIpcMemHandle_t s0 = mine, s1 = mine;
-        if (c->host_exchange(g.nbf[3], g.nbb[3], &s0, &s1, &hb, &hf, sizeof(mine), c->comm_user))
+        Rec s0 = mine, s1 = mine;
+        if (c->host_exchange(g.nbf[3], g.nbb[3], &s0, &s1, &rb, &rf, sizeof(Rec), c->comm_user))
             throw Error(QUDAX_ERR_COMM, "host_exchange hook failed (IPC handles)");
     } else if (c->comm == QUDAX_COMM_NCCL) {
-        char *d = static_cast<char *>(dalloc(c, 3 * sizeof(mine)));
-        QX_CUDA(cudaMemcpyAsync(d, &mine, sizeof(mine), cudaMemcpyHostToDevice, c->stream));
-        exchange(c, d, d, d + 64, d + 128, sizeof(mine), c->stream, nullptr, nullptr, nullptr, nullptr);
-        QX_CUDA(cudaMemcpyAsync(&hb, d + 64, sizeof(mine), cudaMemcpyDeviceToHost, c->stream));
-        QX_CUDA(cudaMemcpyAsync(&hf, d + 128, sizeof(mine), cudaMemcpyDeviceToHost, c->stream));
+        char *d = static_cast<char *>(dalloc(c, 3 * sizeof(Rec)));
+        QX_CUDA(cudaMemcpyAsync(d, &mine, sizeof(Rec), cudaMemcpyHostToDevice, c->stream));
+        exchange(c, d, d, d + sizeof(Rec), d + 2 * sizeof(Rec), sizeof(Rec), c->stream, nullptr, nullptr, nullptr,
+                 nullptr);
+        QX_CUDA(cudaMemcpyAsync(&rb, d + sizeof(Rec), sizeof(Rec), cudaMemcpyDeviceToHost, c->stream));
+        QX_CUDA(cudaMemcpyAsync(&rf, d + 2 * sizeof(Rec), sizeof(Rec), cudaMemcpyDeviceToHost, c->stream));
         QX_CUDA(cudaStreamSynchronize(c->stream));
+        dfree(c, d);
     } else {
         throw Error(QUDAX_ERR_ARG, "P2P halo with nranks > 1 needs a comm transport for the handle exchange");
     }
+    for (const Rec *r : {&rb, &rf}) {
+        if (std::strncmp(r->bus, mine.bus, sizeof(mine.bus)) == 0) continue;  // same GPU (test mode)
+        int peer = -1, can = 0;
+        if (cudaDeviceGetByPCIBusId(&peer, r->bus) != cudaSuccess) {
+            cudaGetLastError();  // the peer GPU is not visible to this process: no peer access
+            throw Error(QUDAX_ERR_UNSUPPORTED, std::string("P2P halo: neighbour GPU ") + r->bus + " not visible here");
+        }
+        QX_CUDA(cudaDeviceCanAccessPeer(&can, c->device, peer));
+        if (!can)
+            throw Error(QUDAX_ERR_UNSUPPORTED, std::string("P2P halo: no peer access to neighbour GPU ") + r->bus);
+    }
+    const cudaIpcMemHandle_t hb = rb.h, hf = rf.h;
     void *pb = nullptr;
     QX_CUDA(cudaIpcOpenMemHandle(&pb, hb, cudaIpcMemLazyEnablePeerAccess));
     q.peer_back = static_cast<char *>(pb);
@@ -1246,10 +1204,8 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         }
         QX_CHECK(g.V < (1L << 30), QUDAX_ERR_ARG, "local volume too large for 32-bit site indexing");
         c->device = p->device;
-        if (const char *ng = std::getenv("QUDAX_NO_GRAPHS")) c->no_graphs = (ng[0] == '1');
-        if (const char *fg = std::getenv("QUDAX_GRAPHS")) c->force_graphs = (fg[0] == '1');
-        if (const char *ds = std::getenv("QUDAX_DEBUG_SOLVER")) c->debug_solver = (ds[0] == '1');
-        if (const char *fu = std::getenv("QUDAX_FUSED")) c->fused = (fu[0] == '1');
+        c->flags = p->flags;
+        if (p->copy_threads > 0 && g_copy_threads == 0) g_copy_threads = p->copy_threads;
         c->comm = p->comm;
         c->overlap = p->overlap;
         c->dev_alloc = p->dev_alloc; c->dev_free = p->dev_free; c->alloc_user = p->alloc_user;
@@ -1275,6 +1231,16 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
         c->red_out = static_cast<double *>(dalloc(c, sizeof(double) * 8));
         c->h_red = static_cast<double *>(halloc(c, sizeof(double) * 8));
         c->d_flag = static_cast<int *>(dalloc(c, sizeof(int) * 4));
+        {  // device error word, readable by the host after any synchronisation without a copy
+            void *h = nullptr;
+            QX_CUDA(cudaHostAlloc(&h, 64, cudaHostAllocMapped));
+            c->host_allocs.push_back(h);
+            c->h_err = static_cast<int *>(h);
+            *c->h_err = 0;
+            void *d = nullptr;
+            QX_CUDA(cudaHostGetDevicePointer(&d, h, 0));
+            c->d_err = static_cast<int *>(d);
+        }
         // reduction tail counters: [0] groups done, [1 + g] CTAs done in group g (reduce.cuh)
         const size_t ncount = 2 + (size_t)(g.Vh / 32) / 64 + 64;
         c->d_counter = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * ncount));
@@ -1314,7 +1280,7 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
 
 qudax_status qudax_finalize(qudax_ctx *c) {
     if (!c) return QUDAX_ERR_ARG;
-    if (g_tbreak_on)
+    if (c->flags & QUDAX_FLAG_TIMING_BREAKDOWN)
         for (auto &kv : g_tbreak)
             std::fprintf(stderr, "qudax timing: prec %d kind %d red %d: %ld launches, %.2f us avg\n", std::get<0>(kv.first),
                          std::get<1>(kv.first), std::get<2>(kv.first), kv.second.first, 1e3 * kv.second.second / kv.second.first);
@@ -1331,6 +1297,7 @@ qudax_status qudax_finalize(qudax_ctx *c) {
     for (void *p : c->host_allocs) cudaFreeHost(p);
     for (auto &r : c->trecs) { cudaEventDestroy(r.a); cudaEventDestroy(r.b); }
     for (auto &r : c->graph_trecs) { cudaEventDestroy(r.a); cudaEventDestroy(r.b); }
+    drop_graphs(c);  // (their timing events go back to the pool, destroyed below)
     for (auto e : c->ev_pool) cudaEventDestroy(e);
     for (auto e : c->xfer.done)
         if (e) cudaEventDestroy(e);
@@ -1349,6 +1316,7 @@ qudax_status qudax_sync(qudax_ctx *c) {
     return guard(c, [&] {
         QX_CUDA(cudaStreamSynchronize(c->stream));
         QX_CUDA(cudaStreamSynchronize(c->comm_stream));
+        check_device_error(c);
     });
 }
 

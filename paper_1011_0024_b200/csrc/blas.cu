@@ -46,9 +46,11 @@ __device__ __forceinline__ void block_reduce_store(double (&v)[NRED], const RedT
 }
 
 // BiCGstab scalar recurrence after a multi-rank allreduce of S->red (single thread)
-__global__ void k_coef(SolverScalars *S, int mode) { apply_coef(S, mode); }
-void launch_coef(SolverScalars *S, int mode, cudaStream_t s) {
-    k_coef<<<1, 1, 0, s>>>(S, mode);
+__global__ void k_coef(SolverScalars *S, int mode, const int *halt) {
+    if (!halted(halt)) apply_coef(S, mode);
+}
+void launch_coef(SolverScalars *S, int mode, const int *halt, cudaStream_t s) {
+    k_coef<<<1, 1, 0, s>>>(S, mode, halt);
     QX_CUDA(cudaGetLastError());
 }
 
@@ -56,7 +58,9 @@ void launch_coef(SolverScalars *S, int mode, cudaStream_t s) {
 
 // p <- r + beta (p - omega v)            (BiCGstab search direction)
 template <int P>
-__global__ void k_p_update(long Vh, long stride, const void *r, void *p, const void *v, CoefArg beta_, CoefArg omega_) {
+__global__ void k_p_update(long Vh, long stride, const void *r, void *p, const void *v, CoefArg beta_, CoefArg omega_,
+                           const int *halt) {
+    if (halted(halt)) return;
     using R = typename Prec<P>::R;
     const double2 beta = coef_get(beta_), omega = coef_get(omega_);
     const Cx<R> b = cx((R)beta.x, (R)beta.y), w = cx((R)omega.x, (R)omega.y);
@@ -78,7 +82,8 @@ __global__ void k_p_update(long Vh, long stride, const void *r, void *p, const v
 
 // y <- y + c x   (c complex)
 template <int P>
-__global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y) {
+__global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y, const int *halt) {
+    if (halted(halt)) return;
     using R = typename Prec<P>::R;
     const double2 c = coef_get(c_);
     const Cx<R> a = cx((R)c.x, (R)c.y);
@@ -98,7 +103,8 @@ __global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y
 
 // z <- x + a y  (real a); z may alias x or y
 template <int P>
-__global__ void k_xpay(long Vh, long stride, const void *x, double a, const void *y, void *z) {
+__global__ void k_xpay(long Vh, long stride, const void *x, double a, const void *y, void *z, const int *halt) {
+    if (halted(halt)) return;
     using R = typename Prec<P>::R;
     QX_GRID_LOOP(i) {
         R xx[24], yy[24];
@@ -112,7 +118,8 @@ __global__ void k_xpay(long Vh, long stride, const void *x, double a, const void
 
 // sum conj(a) b -> (re, im)
 template <int P>
-__global__ void k_cdot(long Vh, long stride, const void *a, const void *b, RedTail tail) {
+__global__ void k_cdot(long Vh, long stride, const void *a, const void *b, RedTail tail, const int *halt) {
+    if (halted(halt)) return;
     using R = typename Prec<P>::R;
     double acc[2] = {0, 0};
     QX_GRID_LOOP(i) {
@@ -130,7 +137,8 @@ __global__ void k_cdot(long Vh, long stride, const void *a, const void *b, RedTa
 
 // sum |a|^2
 template <int P>
-__global__ void k_norm2(long Vh, long stride, const void *a, RedTail tail) {
+__global__ void k_norm2(long Vh, long stride, const void *a, RedTail tail, const int *halt) {
+    if (halted(halt)) return;
     using R = typename Prec<P>::R;
     double acc[1] = {0};
     QX_GRID_LOOP(i) {
@@ -144,7 +152,8 @@ __global__ void k_norm2(long Vh, long stride, const void *a, RedTail tail) {
 
 // (<t, s>, |t|^2)
 template <int P>
-__global__ void k_tdot(long Vh, long stride, const void *t, const void *s, RedTail tail) {
+__global__ void k_tdot(long Vh, long stride, const void *t, const void *s, RedTail tail, const int *halt) {
+    if (halted(halt)) return;
     using R = typename Prec<P>::R;
     double acc[3] = {0, 0, 0};
     QX_GRID_LOOP(i) {
@@ -168,7 +177,8 @@ __global__ void k_tdot(long Vh, long stride, const void *t, const void *s, RedTa
 template <int P>
 __global__ void __launch_bounds__(kBlasThreads, P == 4 ? QX_BICG_MINB : 1)
 k_bicg_final(long Vh, long stride, void *x, const void *p, void *s, const void *t, const void *rhat,
-                             CoefArg alpha_, CoefArg omega_, RedTail tail) {
+                             CoefArg alpha_, CoefArg omega_, RedTail tail, const int *halt) {
+    if (halted(halt)) return;
     using R = typename Prec<P>::R;
     const double2 alpha = coef_get(alpha_), omega = coef_get(omega_);
     const Cx<R> al = cx((R)alpha.x, (R)alpha.y), om = cx((R)omega.x, (R)omega.y);
@@ -176,9 +186,11 @@ k_bicg_final(long Vh, long stride, void *x, const void *p, void *s, const void *
     if constexpr (P == 4) {
         // fp32: one float4 block (two complex components) of all five fields at a time, in the
         // site's component order (so every value and every fp64 partial sum is bitwise the
-        // whole-site version's): ~30 instead of 72 registers, 8 instead of 3 resident 256-thread
-        // CTAs per SM, and the loads of the next block in flight while this one is computed
-        // (the whole-site form was latency-bound at 0.78 of HBM, profiles/r01k_ncu_blas.txt)
+        // whole-site version's): 54 instead of 72 registers, 4 instead of 3 resident 256-thread
+        // CTAs per SM (-Xptxas -v), and the loads of the next block in flight while this one is
+        // computed (the whole-site form was latency-bound at 0.78 of HBM,
+        // profiles/r01k_ncu_blas.txt).  x and s are written by this kernel, so they are read
+        // with plain (coherent) loads; only p, t and rhat take the read-only path.
         QX_GRID_LOOP(i) {
             float4 *X = reinterpret_cast<float4 *>(x);
             float4 *Sv = reinterpret_cast<float4 *>(s);
@@ -187,7 +199,7 @@ k_bicg_final(long Vh, long stride, void *x, const void *p, void *s, const void *
 #pragma unroll
             for (int k = 0; k < 6; ++k) {
                 const long j = (long)k * stride + i;
-                const float4 xv = __ldg(X + j), pv = __ldg(Pp + j), sv = __ldg(Sv + j), tv = __ldg(T + j), hv = __ldg(H + j);
+                const float4 xv = __ldcs(X + j), pv = __ldg(Pp + j), sv = __ldcs(Sv + j), tv = __ldg(T + j), hv = __ldg(H + j);
                 const float xr[4] = {xv.x, xv.y, xv.z, xv.w}, pr[4] = {pv.x, pv.y, pv.z, pv.w};
                 const float sr[4] = {sv.x, sv.y, sv.z, sv.w}, tr[4] = {tv.x, tv.y, tv.z, tv.w};
                 const float hr[4] = {hv.x, hv.y, hv.z, hv.w};
@@ -264,7 +276,8 @@ __global__ void k_xpy_mixed(long Vh, long stride, const void *x, void *y) {
 
 // r <- b - r ; returns |r|^2
 template <int P>
-__global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, RedTail tail) {
+__global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, RedTail tail, const int *halt) {
+    if (halted(halt)) return;
     using R = typename Prec<P>::R;
     double acc[1] = {0};
     QX_GRID_LOOP(i) {
@@ -298,37 +311,38 @@ __global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, RedTail
         K<<<B_, kBlasThreads, 0, s>>>(__VA_ARGS__);    \
     } while (0)
 
-int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail, cudaStream_t s) {
+int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail, const int *halt,
+             cudaStream_t s) {
     const long Vh = g.Vh, st = g.stride;
     int nred = 0;
     switch (op) {
         case OP_P_UPDATE:  // p = r + beta (p - omega v): r=f0, p=f1, v=f2
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_p_update<P>, Vh, st, f[0], f[1], f[2], co[0], co[1]));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_p_update<P>, Vh, st, f[0], f[1], f[2], co[0], co[1], halt));
             break;
         case OP_CAXPY:  // f1 += c f0
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_caxpy<P>, Vh, st, co[0], f[0], f[1]));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_caxpy<P>, Vh, st, co[0], f[0], f[1], halt));
             break;
         case OP_XPAY:  // f2 = f0 + a f1
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_xpay<P>, Vh, st, f[0], co[0].v.x, f[1], f[2]));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_xpay<P>, Vh, st, f[0], co[0].v.x, f[1], f[2], halt));
             break;
         case OP_CDOT:  // <f0, f1>
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_cdot<P>, Vh, st, f[0], f[1], tail));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_cdot<P>, Vh, st, f[0], f[1], tail, halt));
             nred = 2;
             break;
         case OP_NORM2:
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_norm2<P>, Vh, st, f[0], tail));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_norm2<P>, Vh, st, f[0], tail, halt));
             nred = 1;
             break;
         case OP_TDOT:  // (<f0, f1>, |f0|^2)
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_tdot<P>, Vh, st, f[0], f[1], tail));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_tdot<P>, Vh, st, f[0], f[1], tail, halt));
             nred = 3;
             break;
         case OP_FINAL:  // x=f0, p=f1, s=f2, t=f3, rhat=f4
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bicg_final<P>, Vh, st, f[0], f[1], f[2], f[3], f[4], co[0], co[1], tail));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bicg_final<P>, Vh, st, f[0], f[1], f[2], f[3], f[4], co[0], co[1], tail, halt));
             nred = 3;
             break;
         case OP_BMR_NORM:  // f1 = f0 - f1
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bmr_norm<P>, Vh, st, f[0], f[1], tail));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bmr_norm<P>, Vh, st, f[0], f[1], tail, halt));
             nred = 1;
             break;
         default:

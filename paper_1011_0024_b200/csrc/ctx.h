@@ -34,29 +34,38 @@ struct qudax_ctx {
         long sites;
         int nrhs = 1;  // multi-RHS launch: links and clover are compulsory once, spinors per RHS
         int red = 0;   // fused reduction kind (RED_RHAT_DOT reads rhat: +1 spinor per site)
+        int iter = 0;  // graph-captured launches: solver iteration within the batch
     };
     std::vector<TimingRec> trecs;
     std::vector<cudaEvent_t> ev_pool;
     // Dslash launches inside a captured CUDA graph: their (external) events are re-recorded at
     // every replay, so they are harvested into running sums after each replay
     std::vector<TimingRec> graph_trecs;
+    // solver iteration batches captured as CUDA graphs, cached across solves (keyed by every
+    // pointer and parameter the captured launches bake in; gauge_epoch changes on gauge_load)
+    struct Graph {
+        std::vector<uintptr_t> key;
+        cudaGraphExec_t exec = nullptr;
+        long long launches = 0;          // library kernels per replay
+        std::vector<TimingRec> trecs;    // event-bracketed Dslash launches (kernel timing on)
+    };
+    std::vector<Graph> graphs;
+    long long gauge_epoch = 0;
     struct TimingAcc {
         long long launches = 0, sites = 0;
         double ms = 0, flops = 0, bytes_c = 0, bytes_p = 0;
     } tacc[3];
     bool capturing = false;
-    bool no_graphs = false;   // QUDAX_NO_GRAPHS=1: eager solver iterations (debug / comparison)
-    bool force_graphs = false;  // QUDAX_GRAPHS=1: graph replay also with nranks > 1
-    bool debug_solver = false;  // QUDAX_DEBUG_SOLVER=1: per-iteration scalars to stderr
-    // single-launch wavefront Mhat on unpartitioned contexts (QUDAX_FUSED=1).  Off by default:
-    // measured slower than the two kernels (L2 kept only ~1/3 of the reusable bytes, plus
-    // dependency waits) — profiles/r01_fused_matpc.md
-    bool fused = false;
+    int cap_iter = 0;           // solver iteration (within the captured batch) being captured
+    int flags = 0;              // qudax_init_flag bits
+    // solver batch gate: while set, every kernel the library launches carries this pointer
+    // (SolverScalars::halt) and returns at once when an earlier iteration set it
+    const int *halt = nullptr;
+    // device error word in mapped pinned host memory (kernel-initiated halo wait timeout)
+    int *h_err = nullptr, *d_err = nullptr;
     // the Schur form matpc_op applies: 0 asymmetric (default), 1 symmetric (set by a solve with
     // use_schur = 2 for its duration, and by qudax_matpc_sym)
     int matpc_sym = 0;
-    const int *fstages = nullptr;
-    unsigned *fcounters = nullptr;
     qx::SolverScalars *d_scal = nullptr, *h_scal = nullptr;
     std::vector<void *> allocs;       // device allocations owned by the ctx
     std::vector<void *> host_allocs;  // pinned host allocations
@@ -135,6 +144,7 @@ namespace qx {
 inline int prec_idx(int prec) { return prec == 8 ? 0 : (prec == 4 ? 1 : 2); }
 void *dalloc(qudax_ctx *c, size_t bytes);
 void *halloc(qudax_ctx *c, size_t bytes);
+void dfree(qudax_ctx *c, void *p);  // releases a dalloc'ed buffer (no-op for nullptr)
 void check_prec(int prec);
 // optional reduction fused into a Dslash epilogue (see DslashRed); res: 3 global sums (host)
 struct RedReq {
@@ -164,6 +174,10 @@ void xpy_mixed_op(qudax_ctx *c, int pd, int ps, const void *x, void *y);
 void convert_op(qudax_ctx *c, void *dst, int pd, const void *src, int ps);
 void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *p, qudax_solve_stats *st);
 void cgnr_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solve_param *p, qudax_solve_stats *st);
-void harvest_graph_timing(qudax_ctx *c);
-void release_graph_timing(qudax_ctx *c);
+void harvest_graph_timing(qudax_ctx *c, const std::vector<qudax_ctx::TimingRec> &recs, int iters);
+void release_graph_timing(qudax_ctx *c, std::vector<qudax_ctx::TimingRec> &recs);
+// destroy the cached solver graphs (gauge_load: they baked in the old gauge / clover)
+void drop_graphs(qudax_ctx *c);
+// raise QUDAX_ERR_COMM if a kernel set the device error word (call after a synchronisation)
+void check_device_error(qudax_ctx *c);
 }  // namespace qx

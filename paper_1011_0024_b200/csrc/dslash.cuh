@@ -814,9 +814,11 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
 }
 
 // Kernel-initiated halo (QUDAX_HALO_P2P): one thread per CTA acquires the two flags the
-// neighbours raise after storing this sequence number's faces into our ghosts (bounded: a
-// broken protocol surfaces as a wrong result, never a hang).  Returns the ghost byte offset of
-// the sequence parity.
+// neighbours raise after storing this sequence number's faces into our ghosts.  The wait is
+// bounded (a stalled neighbour must not hang the GPU): on timeout the CTA raises the context's
+// device error word, which the host checks at its next synchronisation and reports as
+// QUDAX_ERR_COMM instead of returning an operator applied to stale ghosts.  Returns the ghost
+// byte offset of the sequence parity.
 __device__ __forceinline__ unsigned ld_acquire_sys(const unsigned *p) {
     unsigned v;
     asm volatile("ld.acquire.sys.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
@@ -826,10 +828,12 @@ __device__ __forceinline__ long p2p_wait(const DslashArgs &a) {
     __shared__ unsigned s_seq;
     if (threadIdx.x == 0) {
         const unsigned s = *reinterpret_cast<const volatile unsigned *>(a.p2p_cseq) + 1u;
-        for (long spin = 0; spin < (1L << 28); ++spin) {
-            if ((int)(ld_acquire_sys(a.p2p_flags) - s) >= 0 && (int)(ld_acquire_sys(a.p2p_flags + 1) - s) >= 0) break;
-            __nanosleep(128);
+        bool ok = false;
+        for (long spin = 0; spin < (1L << 24) && !ok; ++spin) {  // >= 2 s of 128 ns sleeps
+            ok = (int)(ld_acquire_sys(a.p2p_flags) - s) >= 0 && (int)(ld_acquire_sys(a.p2p_flags + 1) - s) >= 0;
+            if (!ok) __nanosleep(128);
         }
+        if (!ok && a.err) atomicExch(a.err, 1);
         s_seq = s;
     }
     __syncthreads();
@@ -842,6 +846,7 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     // hardware CTA scheduler balances the memory-latency-bound CTAs better than a fixed wave)
     // multi-RHS (a.nrhs > 1): consecutive CTAs take the same sites for different right-hand
     // sides, so the links and clover they stream are served from L2 after the first of them
+    if (halted(a.halt)) return;  // the rest of a solver batch after a reliable-update request
     int blk = blockIdx.x, rhs = 0;
     if (a.nrhs > 1) {
         rhs = blk % a.nrhs;
@@ -897,8 +902,7 @@ void launch_dslash_prec(int recon, int dagger, int kind, const DslashArgs &a, cu
     const int threads = QX_DSLASH_THREADS;
     if (a.nthreads <= 0) return;
     if constexpr (P != 8 && !SS) {  // several right-hand sides per thread (dslash_mr.cuh)
-        static const bool mr_off = std::getenv("QUDAX_MR_OFF") != nullptr;  // A/B: one RHS per thread
-        if (a.nrhs > 1 && !mr_off &&
+        if (a.nrhs > 1 && !(a.variant & kVariantOneRhsPerThread) &&
             (P == 4 ? launch_dslash_mr_f32(recon, dagger, kind, a, s) : launch_dslash_mr_f16(recon, dagger, kind, a, s)))
             return;
     }

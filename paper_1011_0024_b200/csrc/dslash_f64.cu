@@ -1,22 +1,15 @@
 // dslash_f64.cu — instantiation of the Dslash kernel family for storage precision 8 bytes/real
 // (split per precision so the 18 variants per precision compile in parallel).
-#include <cstdlib>
-
 #include "dslash.cuh"
-#include "matpc_fused.cuh"
 
 namespace qx {
 void launch_dslash_f64_ss(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
 void launch_dslash_f64(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
-    static const bool force_ss = std::getenv("QUDAX_FORCE_SS") != nullptr;  // debug: SS variant everywhere
-    if (a.smask || force_ss) launch_dslash_f64_ss(recon, dagger, kind, a, s);  // partitioned X / Y / Z
+    // partitioned X / Y / Z, or the test flag that runs that instantiation everywhere
+    if (a.smask || (a.variant & kVariantForceSS)) launch_dslash_f64_ss(recon, dagger, kind, a, s);  // partitioned X / Y / Z
     else launch_dslash_prec<8>(recon, dagger, kind, a, s);
 }
 int dslash_blocks_f64(int recon, int dagger, int kind, int nthreads) {
     return dslash_blocks_prec<8>(recon, dagger, kind, nthreads);
 }
-void launch_matpc_fused_f64(int recon, int dagger, const FusedArgs &f, int grid, cudaStream_t s) {
-    launch_matpc_fused_prec<8>(recon, dagger, f, grid, s);
-}
-int matpc_fused_wave_f64(int recon, int dagger) { return matpc_fused_wave<8>(recon, dagger); }
 }  // namespace qx

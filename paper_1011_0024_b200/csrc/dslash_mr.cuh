@@ -292,6 +292,7 @@ __device__ __forceinline__ void dslash_site_mr(const DslashArgs &a, int tid, con
 // grid: (site blocks) x (RHS groups of NR), consecutive CTAs = the groups of one site block
 template <int P, int RECON, bool DAG, int KIND, int NR>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, DslashMrMinBlocks<P, NR>::value) dslash_mr_kernel(const __grid_constant__ DslashArgs a) {
+    if (halted(a.halt)) return;
     const int ng = (a.nrhs + NR - 1) / NR;
     const int grp = blockIdx.x % ng, blk = blockIdx.x / ng;
     const int r0 = grp * NR;

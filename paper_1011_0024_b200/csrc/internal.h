@@ -81,10 +81,26 @@ inline int spatial_split(const Geom &g) { return g.split & 7; }
 
 // ----------------------------------------------------------------------------- reductions
 // device-resident BiCGstab scalars (Algorithm R), advanced by apply_coef after each reduction
+// The iteration's update rule (Algorithm R, solver.cpp) is evaluated on the device right after
+// the |r|^2 reduction (COEF_RHO with decide != 0): the host reads the scalars once per batch of
+// `poll_every` iterations instead of after every iteration.  An iteration that calls for a
+// reliable update sets `halt`; every kernel launched for the rest of the batch (they carry a
+// pointer to it) returns at once, so the iterates are exactly those of a host decision taken
+// after every iteration.
+constexpr int kHistRing = 64;  // per-iteration |r| of the current batch (poll_every <= kHistRing)
 struct SolverScalars {
     double2 rho, rho_new, alpha, malpha, omega, beta;
     double r2;
     double red[3];
+    // Algorithm R state advanced on the device (decide != 0)
+    double rNorm, r0Norm, maxrr, maxrx;
+    double delta, stop;          // update threshold, tol * ||bhat||
+    int k, maxiter;              // iterations done in this solve, cap
+    int decide;                  // evaluate the update rule after COEF_RHO
+    int halt;                    // an iteration of this batch asked for a reliable update
+    int updX, blown;             // its flags (reading R3 for blown)
+    int pad_;
+    double hist[kHistRing];      // |r_k| (iterated) at ring slot (k - 1) % kHistRing
 };
 enum CoefMode { COEF_NONE = 0, COEF_ALPHA = 1, COEF_OMEGA = 2, COEF_RHO = 3 };
 // a grid reduction with a last-CTA tail (reduce.cuh)
@@ -175,6 +191,9 @@ struct DslashArgs {
     RedTail tail;          // 3 sums per CTA; block_offset set per launch (split launches)
     const void *rhat;
     int reverse;           // 1: map CTAs to sites from the top of the range down (L2 reuse, see matpc)
+    const int *halt;       // solver batch gate (SolverScalars::halt), nullptr outside solver batches
+    int *err;              // device error word (kernel-initiated halo wait timeout -> QUDAX_ERR_COMM)
+    int variant;           // kVariant* bits (init flags: test / comparison instantiations)
     // multi-RHS launch: nrhs > 1 uses in_m / out_m / x_m instead of in/out/x
     int nrhs;
     const void *in_m[kMaxRhs];
@@ -186,22 +205,8 @@ struct DslashArgs {
     RedTail tail_m[kMaxRhs];
 };
 enum DslashRed { RED_NONE = 0, RED_XDOT_NORM = 1, RED_RHAT_DOT = 2 };
+enum DslashVariant { kVariantForceSS = 1, kVariantOneRhsPerThread = 2 };
 
-// single-launch Mhat (matpc_fused.cuh): phase A = CLOVER_INV on odd, phase B = CLOVER_XPAY on even
-struct FusedArgs {
-    DslashArgs A, B;
-    int chunks;           // work items per timeslice and phase: ceil(F / threads)
-    int total_items;      // 2 T_loc chunks
-    const int *stages;    // [2 T_loc] dispense order: t (phase A) or T_loc + t (phase B)
-    unsigned *work;       // item counter, zero on entry
-    unsigned *doneA;      // [T_loc] completed phase-A chunks per timeslice, zero on entry
-};
-void launch_matpc_fused_f64(int recon, int dagger, const FusedArgs &f, int grid, cudaStream_t s);
-void launch_matpc_fused_f32(int recon, int dagger, const FusedArgs &f, int grid, cudaStream_t s);
-void launch_matpc_fused_f16(int recon, int dagger, const FusedArgs &f, int grid, cudaStream_t s);
-int matpc_fused_wave_f64(int recon, int dagger);
-int matpc_fused_wave_f32(int recon, int dagger);
-int matpc_fused_wave_f16(int recon, int dagger);
 
 void launch_dslash_f64(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
 void launch_dslash_f32(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s);
@@ -215,7 +220,7 @@ int dslash_blocks_f16(int recon, int dagger, int kind, int nthreads);
 // x_mu = 0 face projected with the receiver's forward-hop projector -> sb[mu], the x_mu = L-1
 // face with its backward-hop projector -> sf[mu]; 12 reals per site in the arithmetic precision
 void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, const void *in, void *const sb[3],
-                         void *const sf[3], cudaStream_t s);
+                         void *const sf[3], const int *halt, cudaStream_t s);
 // whether the faces along mu carry raw spinor records (half everywhere; X in every precision)
 // instead of spin-projected half spinors in the arithmetic precision
 __host__ __device__ inline bool sface_raw(int prec, int mu) { return prec == 2 || mu == 0; }
@@ -224,14 +229,14 @@ size_t sface_bytes(int prec, int mu, long fs);
 // face pack: t_loc = 0 slice half (lower if !dagger) -> send_back; t_loc = T_loc-1 half
 // (upper if !dagger) -> send_fwd.  `in` is the Dslash input field (parity 1-p).
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back,
-                       void *send_fwd, cudaStream_t s);
+                       void *send_fwd, const int *halt, cudaStream_t s);
 // kernel-initiated halo (QUDAX_HALO_P2P): the same faces stored straight into the neighbours'
 // ghost buffers dst_back / dst_fwd (+ pdist bytes for odd sequence numbers), then flag_back /
 // flag_fwd (in the neighbours' memory) set to the new sequence number with a system-scope
 // release.  seq / count: this rank's sequence counter and CTA counter (device).
 void launch_pack_faces_p2p(int prec, int dagger, const Geom &g, const void *in, char *dst_back, char *dst_fwd,
                            size_t pdist, unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count,
-                           cudaStream_t s);
+                           const int *halt, cudaStream_t s);
 
 // layout conversion (DR AoS fp64 <-> NR SoA prec), one parity
 void launch_spinor_import(int prec, const Geom &g, int parity, const double *src, void *dst, cudaStream_t s);
@@ -273,8 +278,16 @@ __device__ __forceinline__ double2 coef_get(const CoefArg &c) { return c.d ? *c.
 #endif
 // `tail` describes the reduction of reducing ops (partials/counter/out/S/coef_mode; the
 // block fields are filled in here).  Returns the number of reduced doubles (0 if none).
-int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail, cudaStream_t s);
-void launch_coef(SolverScalars *S, int mode, cudaStream_t s);
+int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail, const int *halt,
+             cudaStream_t s);
+#ifdef __CUDACC__
+// a kernel launched inside a solver batch returns at once once an earlier iteration has asked
+// for a reliable update (SolverScalars::halt); halt == nullptr outside solver batches
+__device__ __forceinline__ bool halted(const int *halt) {
+    return halt && *reinterpret_cast<const volatile int *>(halt);
+}
+#endif
+void launch_coef(SolverScalars *S, int mode, const int *halt, cudaStream_t s);
 void blas_xpy_mixed(int pd, int ps, const Geom &g, const void *x, void *y, cudaStream_t s);
 int blas_partial_blocks();
 

@@ -586,7 +586,8 @@ __device__ __forceinline__ void k_pack_faces_body(long F, long T_loc, long strid
 }
 template <int P>
 __global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
-                             const void *__restrict__ in, void *__restrict__ sb, void *__restrict__ sf) {
+                             const void *__restrict__ in, void *__restrict__ sb, void *__restrict__ sf, const int *halt) {
+    if (halted(halt)) return;
     k_pack_faces_body<P>(F, T_loc, stride, fstride, half_back, half_fwd, in, sb, sf);
 }
 
@@ -600,8 +601,13 @@ __device__ __forceinline__ void st_release_sys(unsigned *p, unsigned v) {
 template <int P>
 __global__ void k_pack_faces_p2p(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
                                  const void *__restrict__ in, char *dst_back, char *dst_fwd, long pdist,
-                                 unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count) {
+                                 unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count,
+                                 const int *halt) {
     __shared__ bool last;
+    // a halted solver iteration (every rank halts the same one: the decision is taken on
+    // globally summed scalars) skips both the pack and the consuming Dslash, so producer and
+    // consumer sequence counters stay in step
+    if (halted(halt)) return;
     const unsigned s = *reinterpret_cast<volatile unsigned *>(seq) + 1u;
     const long off = (s & 1u) ? pdist : 0L;
     k_pack_faces_body<P>(F, T_loc, stride, fstride, half_back, half_fwd, in, dst_back + off, dst_fwd + off);
@@ -622,14 +628,14 @@ __global__ void k_pack_faces_p2p(long F, long T_loc, long stride, long fstride, 
 
 void launch_pack_faces_p2p(int prec, int dagger, const Geom &g, const void *in, char *dst_back, char *dst_fwd,
                            size_t pdist, unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count,
-                           cudaStream_t s) {
+                           const int *halt, cudaStream_t s) {
     const int half_back = dagger ? 0 : 1;
     const int half_fwd = dagger ? 1 : 0;
     const int T = 128;
     const int b = nblk(2 * g.F, T);
 #define QX_PP(P)                                                                                                \
     k_pack_faces_p2p<P><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, dst_back,   \
-                                        dst_fwd, (long)pdist, flag_back, flag_fwd, seq, count)
+                                        dst_fwd, (long)pdist, flag_back, flag_fwd, seq, count, halt)
     if (prec == 8) QX_PP(8);
     else if (prec == 4) QX_PP(4);
     else QX_PP(2);
@@ -653,10 +659,12 @@ struct SPackArgs {
     int q;          // parity of the packed (input) field
     long Fd[3], fsd[3], stride;
     void *sb[3], *sf[3];
+    const int *halt;
 };
 template <int P, bool DAG>
 __global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *__restrict__ in) {
     using R = typename Prec<P>::R;
+    if (halted(a.halt)) return;
     long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
     int mu = 0;
     for (; mu < 3; ++mu) {
@@ -708,8 +716,9 @@ __global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *
 size_t sface_bytes(int prec, int mu, long fs) { return sface_raw(prec, mu) ? spinor_bytes(prec, fs) : (size_t)12 * prec * fs; }
 
 void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, const void *in, void *const sb[3],
-                         void *const sf[3], cudaStream_t s) {
+                         void *const sf[3], const int *halt, cudaStream_t s) {
     SPackArgs a{};
+    a.halt = halt;
     long n = 0;
     for (int m = 0; m < 4; ++m) a.L[m] = g.L[m];
     a.mask = spatial_split(g);
@@ -738,7 +747,7 @@ void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, con
 }
 
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back, void *send_fwd,
-                       cudaStream_t s) {
+                       const int *halt, cudaStream_t s) {
     // non-dagger: the receiver's forward hop (1 - gamma_4) needs LOWER spins of our t=0 slice
     // (sent backward); its backward hop (1 + gamma_4) needs UPPER spins of our t=T_loc-1 slice
     // (sent forward).  The dagger swaps the halves (reading Q15).
@@ -746,9 +755,9 @@ void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void
     const int half_fwd = dagger ? 1 : 0;
     const int T = 128;
     const int b = nblk(2 * g.F, T);
-    if (prec == 8) k_pack_faces<8><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
-    else if (prec == 4) k_pack_faces<4><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
-    else k_pack_faces<2><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
+    if (prec == 8) k_pack_faces<8><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd, halt);
+    else if (prec == 4) k_pack_faces<4><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd, halt);
+    else k_pack_faces<2><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd, halt);
     QX_CUDA(cudaGetLastError());
 }
 

@@ -37,6 +37,27 @@ __device__ __forceinline__ void apply_coef(SolverScalars *S, int mode) {
         S->rho = S->rho_new;
         S->rho_new = make_double2(r[1], r[2]);
         S->beta = cmul(cdiv(S->rho_new, S->rho), cdiv(S->alpha, S->omega));
+        if (S->decide) {
+            // Algorithm R's update rule (solver.cpp header), the same comparisons in the same
+            // order as the host-side version it replaces
+            const double rn = sqrt(S->r2);
+            S->k += 1;
+            S->hist[(S->k - 1) % kHistRing] = rn;
+            S->rNorm = rn;
+            const bool blown = !isfinite(rn) || rn > 1e2 * S->maxrr;  // reading R3
+            if (!blown) {
+                if (rn > S->maxrx) S->maxrx = rn;
+                if (rn > S->maxrr) S->maxrr = rn;
+            }
+            const bool updX = !blown && (rn < S->delta * S->r0Norm) && (S->r0Norm <= S->maxrx);
+            const bool updR = blown || ((rn < S->delta * S->maxrr) && (S->r0Norm <= S->maxrr)) || updX ||
+                              (rn <= S->stop) || (S->k >= S->maxiter);
+            if (updR) {
+                S->updX = updX;
+                S->blown = blown;
+                S->halt = 1;
+            }
+        }
     }
 }
 

@@ -23,7 +23,8 @@
 #include <complex>
 #include <cstdio>
 #include <cstring>
-#include <map>
+#include <string>
+#include <vector>
 
 #include "ctx.h"
 
@@ -34,6 +35,26 @@ using cd = std::complex<double>;
 static void *field(qudax_ctx *c, void *&slot, int prec) {
     if (!slot) slot = dalloc(c, spinor_bytes(prec, c->g.stride));
     return slot;
+}
+
+// Point a solver workspace at (Pd, Ps): the fields of a precision that changes are released
+// (the outer-precision fields survive a change of the sloppy precision alone), so switching
+// modes never strands device memory until finalize.
+static void ws_select(qudax_ctx *c, qudax_ctx::SolverWs &w, int Pd, int Ps) {
+    if (w.prec != Pd) {
+        for (void **f : {&w.b_e, &w.b_o, &w.bh, &w.x_e, &w.x_o, &w.r, &w.t_e, &w.t_o}) {
+            dfree(c, *f);
+            *f = nullptr;
+        }
+        w.prec = Pd;
+    }
+    if (w.prec_s != Ps) {
+        for (void **f : {&w.rs, &w.xs, &w.p, &w.v, &w.t, &w.r0}) {
+            dfree(c, *f);
+            *f = nullptr;
+        }
+        w.prec_s = Ps;
+    }
 }
 
 static void zero(qudax_ctx *c, void *f, int prec) {
@@ -65,30 +86,75 @@ static SolverScalars *scalars(qudax_ctx *c) {
 }
 
 // Capture `body` (stream-ordered work on c->stream, possibly forking to the comm stream for
-// the NCCL halo) into an instantiated CUDA graph.  *nlaunch = library kernels per replay.
+// the NCCL halo) into an instantiated CUDA graph.  *nlaunch = library kernels per replay;
+// *trecs receives the event-bracketed Dslash launches (kernel timing on).
 template <typename F>
-static cudaGraphExec_t capture_graph(qudax_ctx *c, F &&body, long long *nlaunch) {
+static cudaGraphExec_t capture_graph(qudax_ctx *c, F &&body, long long *nlaunch,
+                                     std::vector<qudax_ctx::TimingRec> *trecs) {
     const long long l0 = c->launches;
     c->capturing = true;
+    c->graph_trecs.clear();
     QX_CUDA(cudaStreamBeginCapture(c->stream, cudaStreamCaptureModeThreadLocal));
     try {
         body();
     } catch (...) {
         cudaGraph_t g;
         cudaStreamEndCapture(c->stream, &g);
+        if (g) cudaGraphDestroy(g);
         c->capturing = false;
+        c->cap_iter = 0;
+        release_graph_timing(c, c->graph_trecs);
         throw;
     }
     cudaGraph_t graph;
     QX_CUDA(cudaStreamEndCapture(c->stream, &graph));
     c->capturing = false;
+    c->cap_iter = 0;
     cudaGraphExec_t exec;
     QX_CUDA(cudaGraphInstantiate(&exec, graph, 0));
     cudaGraphDestroy(graph);
     *nlaunch = c->launches - l0;
     c->launches = l0;
+    trecs->swap(c->graph_trecs);
+    c->graph_trecs.clear();
     return exec;
 }
+
+// Cached solver graphs (ctx.h Graph): at most kMaxGraphs, least recently captured dropped first;
+// all of them on gauge_load (their key holds the gauge epoch).
+constexpr size_t kMaxGraphs = 24;
+void drop_graphs(qudax_ctx *c) {
+    for (auto &gr : c->graphs) {
+        if (gr.exec) cudaGraphExecDestroy(gr.exec);
+        release_graph_timing(c, gr.trecs);
+    }
+    c->graphs.clear();
+}
+template <typename F>
+static qudax_ctx::Graph &cached_graph(qudax_ctx *c, std::vector<uintptr_t> key, F &&body) {
+    key.push_back((uintptr_t)c->gauge_epoch);
+    key.push_back((uintptr_t)c->timing);
+    for (auto &gr : c->graphs)
+        if (gr.key == key) return gr;
+    if (c->graphs.size() >= kMaxGraphs) {
+        auto &old = c->graphs.front();
+        if (old.exec) cudaGraphExecDestroy(old.exec);
+        release_graph_timing(c, old.trecs);
+        c->graphs.erase(c->graphs.begin());
+    }
+    qudax_ctx::Graph gr;
+    gr.key = std::move(key);
+    gr.exec = capture_graph(c, body, &gr.launches, &gr.trecs);
+    c->graphs.push_back(std::move(gr));
+    return c->graphs.back();
+}
+
+// RAII: kernels launched while this is alive carry the solver batch gate
+struct HaltGate {
+    qudax_ctx *c;
+    HaltGate(qudax_ctx *c_, const int *h) : c(c_) { c->halt = h; }
+    ~HaltGate() { c->halt = nullptr; }
+};
 
 // the Schur form matpc_op applies during one solve (restored on every exit path)
 struct SchurForm {
@@ -172,13 +238,9 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     QX_CHECK(sp->maxiter >= 0 && sp->tol >= 0 && sp->delta >= 0, QUDAX_ERR_ARG, "solve: bad parameters");
     std::memset(st, 0, sizeof(*st));
     auto &w = c->sws;
-    if (w.prec != Pd || w.prec_s != Ps) {
-        w = qudax_ctx::SolverWs{};  // (old buffers stay owned by the ctx until finalize)
-        w.prec = Pd;
-        w.prec_s = Ps;
-    }
+    QX_CUDA(cudaStreamSynchronize(c->stream));  // (released buffers may be in flight)
+    ws_select(c, w, Pd, Ps);
     const Geom &g = c->g;
-    const double kappa = c->kappa;
     void *b_e = field(c, w.b_e, Pd), *b_o = field(c, w.b_o, Pd), *bh = field(c, w.bh, Pd);
     void *x_e = field(c, w.x_e, Pd), *x_o = field(c, w.x_o, Pd), *r = field(c, w.r, Pd);
     void *t_e = field(c, w.t_e, Pd), *t_o = field(c, w.t_o, Pd);
@@ -198,20 +260,26 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     copy(c, r, bh, Pd);
     convert_op(c, rs, Ps, r, Pd);
     copy(c, r0, rs, Ps);
-    double rNorm = bnorm;
-    double r0Norm = rNorm, maxrr = rNorm, maxrx = rNorm;
     // device-resident scalars: the iteration needs no host round trip (the coefficient
-    // recurrences run in tiny kernels after each fused reduction)
+    // recurrences and Algorithm R's update rule run in the reduction tails)
     SolverScalars *S = scalars(c);
-    SolverScalars h0{};
+    SolverScalars *hS = c->h_scal;  // pinned staging (written only after a synchronisation)
+    const int poll = sp->poll_every > 0 ? sp->poll_every : 4;
+    QX_CHECK(poll <= kHistRing, QUDAX_ERR_ARG, "poll_every must be <= " + std::to_string(kHistRing));
     {
         const cd rn = cdot_of(c, Ps, r0, rs);
-        h0.rho = make_double2(1, 0);
-        h0.rho_new = make_double2(rn.real(), rn.imag());
-        h0.alpha = make_double2(1, 0);
-        h0.omega = make_double2(1, 0);
-        h0.beta = make_double2(0, 0);  // first iteration: p = rs + 0 * (p - omega v) = rs
-        QX_CUDA(cudaMemcpyAsync(S, &h0, sizeof(h0), cudaMemcpyHostToDevice, c->stream));
+        std::memset(hS, 0, sizeof(*hS));
+        hS->rho = make_double2(1, 0);
+        hS->rho_new = make_double2(rn.real(), rn.imag());
+        hS->alpha = make_double2(1, 0);
+        hS->omega = make_double2(1, 0);
+        hS->beta = make_double2(0, 0);  // first iteration: p = rs + 0 * (p - omega v) = rs
+        hS->rNorm = hS->r0Norm = hS->maxrr = hS->maxrx = bnorm;
+        hS->delta = sp->delta;
+        hS->stop = stop;
+        hS->maxiter = sp->maxiter;
+        hS->decide = 1;
+        QX_CUDA(cudaMemcpyAsync(S, hS, sizeof(*hS), cudaMemcpyHostToDevice, c->stream));
     }
     int k = 0, updates = 0, restarts = 0;
     bool converged = (bnorm == 0.0);
@@ -222,7 +290,8 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     const double matpc_flops = mm.flops * V_h_all;
     const double blas_flops_iter = 960.0 * V_h_all;  // reading Q16 (fused BLAS per iteration)
 
-    // one BiCGstab iteration, fully stream-ordered; its scalars stay on the device
+    // one BiCGstab iteration, fully stream-ordered; its scalars stay on the device and every
+    // kernel is gated on S->halt (HaltGate), so the tail of a batch after an update request is void
     auto enqueue_iteration = [&] {
         {
             void *f[3] = {rs, p, v};
@@ -241,100 +310,109 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
         {
             void *f[5] = {xs, p, rs, t, r0};
             CoefArg co[2] = {{{0, 0}, &S->alpha}, {{0, 0}, &S->omega}};
-            blas_op_dev(c, OP_FINAL, Ps, f, co, S, COEF_RHO);          // x += a p + w s; r = s - w t; rho', beta
+            blas_op_dev(c, OP_FINAL, Ps, f, co, S, COEF_RHO);          // x += a p + w s; r = s - w t; rho', beta; decide
         }
-        QX_CUDA(cudaMemcpyAsync(c->h_scal, S, sizeof(SolverScalars), cudaMemcpyDeviceToHost, c->stream));
     };
-    // Replay the iteration as one CUDA graph (no per-kernel launch latency, no host syncs
-    // inside the iteration).  Not possible with the host transport (its hooks run on the host).
-    // Multi-rank NCCL runs replay eagerly unless QUDAX_GRAPHS=1: graph capture of NCCL p2p is
-    // exercised here only through the N=1 loopback (a single GPU is all this harness has).
-    const bool use_graph = (c->comm != QUDAX_COMM_HOST) && !c->no_graphs && (c->g.nranks == 1 || c->force_graphs);
-    cudaGraphExec_t gexec = nullptr;
-    long long graph_launches = 0;
+    auto enqueue_batch = [&](int n) {
+        HaltGate gate(c, &S->halt);
+        for (int j = 0; j < n; ++j) {
+            c->cap_iter = j;
+            enqueue_iteration();
+        }
+        c->cap_iter = 0;
+    };
+    // Replay batches of `poll` iterations as one CUDA graph (no per-kernel launch latency, no
+    // host synchronisation inside a batch), cached across solves.  Not with the host transport
+    // (its hooks run on the host and synchronise), which polls after every iteration.
+    const bool host_comm = (c->comm == QUDAX_COMM_HOST);
+    const bool use_graph = !host_comm && !(c->flags & QUDAX_FLAG_NO_GRAPHS);
+    const int batch = host_comm ? 1 : poll;
+    bool first = true;
 
     while (!converged && k < sp->maxiter) {
-        if (!use_graph || k == 0) {
-            enqueue_iteration();  // the first iteration runs eagerly (allocates lazily-created buffers)
+        const std::vector<qudax_ctx::TimingRec> *grecs = nullptr;
+        if (!use_graph || first) {
+            // eager (the first batch runs eagerly: it allocates the lazily-created buffers)
+            enqueue_batch(first ? 1 : batch);
+            first = false;
         } else {
-            if (!gexec) gexec = capture_graph(c, enqueue_iteration, &graph_launches);
-            QX_CUDA(cudaGraphLaunch(gexec, c->stream));
-            c->launches += graph_launches;
+            const std::vector<uintptr_t> key = {1, (uintptr_t)Pd, (uintptr_t)Ps, (uintptr_t)batch, (uintptr_t)rs,
+                                                (uintptr_t)xs, (uintptr_t)p, (uintptr_t)v, (uintptr_t)t,
+                                                (uintptr_t)r0, (uintptr_t)S, (uintptr_t)c->matpc_sym};
+            auto &gr = cached_graph(c, key, [&] { enqueue_batch(batch); });
+            QX_CUDA(cudaGraphLaunch(gr.exec, c->stream));
+            c->launches += gr.launches;
+            grecs = &gr.trecs;
         }
+        QX_CUDA(cudaMemcpyAsync(hS, S, sizeof(*hS), cudaMemcpyDeviceToHost, c->stream));
         QX_CUDA(cudaStreamSynchronize(c->stream));
-        harvest_graph_timing(c);
-        const SolverScalars &hs = *c->h_scal;
-        if (c->debug_solver)
-            std::fprintf(stderr, "qudax it %d: r2 %.6e rho (%.4e,%.4e) alpha (%.4e,%.4e) omega (%.4e,%.4e) beta (%.4e,%.4e) red %.4e %.4e %.4e\n",
-                         k, hs.r2, hs.rho_new.x, hs.rho_new.y, hs.alpha.x, hs.alpha.y, hs.omega.x, hs.omega.y,
-                         hs.beta.x, hs.beta.y, hs.red[0], hs.red[1], hs.red[2]);
-        double rNorm_it = std::sqrt(hs.r2);
-        // breakdown guard (reading R3): a non-finite or exploded iterated residual means the
-        // low-precision recurrences hit a (near) Lanczos breakdown.  Recompute the true
-        // residual (dropping xs if it is not finite) and restart the Krylov space from it.
-        const bool blown = !std::isfinite(rNorm_it) || rNorm_it > 1e2 * maxrr;
-        rNorm = rNorm_it;
-        ++k;
-        flops += 2 * matpc_flops + blas_flops_iter;
-        if (!blown) {
-            if (rNorm > maxrx) maxrx = rNorm;
-            if (rNorm > maxrr) maxrr = rNorm;
+        check_device_error(c);
+        const SolverScalars &hs = *hS;
+        const int ran = hs.k - k;  // iterations of this batch that ran (the rest were halted)
+        if (grecs) harvest_graph_timing(c, *grecs, ran);
+        for (int j = 0; j < ran; ++j) {
+            const int kk = k + j + 1;  // 1-based iteration number
+            const double rn = hs.hist[(kk - 1) % kHistRing];
+            if (c->flags & QUDAX_FLAG_DEBUG_SOLVER)
+                std::fprintf(stderr, "qudax it %d: |r| %.6e rho (%.4e,%.4e) alpha (%.4e,%.4e) omega (%.4e,%.4e)\n",
+                             kk - 1, rn, hs.rho_new.x, hs.rho_new.y, hs.alpha.x, hs.alpha.y, hs.omega.x, hs.omega.y);
+            if (sp->res_history && kk - 1 < sp->history_cap) sp->res_history[kk - 1] = bnorm > 0 ? rn / bnorm : 0.0;
+            flops += 2 * matpc_flops + blas_flops_iter;
         }
-        const bool updX = !blown && (rNorm < sp->delta * r0Norm) && (r0Norm <= maxrx);
-        const bool updR = blown || ((rNorm < sp->delta * maxrr) && (r0Norm <= maxrr)) || updX || (rNorm <= stop) ||
-                          (k == sp->maxiter);
-        if (updR) {
-            if (std::isfinite(rNorm_it)) xpy_mixed_op(c, Pd, Ps, xs, x_e);   // x += xs
-            zero(c, xs, Ps);
-            matpc_op(c, r, x_e, Pd, 0);          // r = Mhat x (high)
-            double r2;
-            {
-                void *f[2] = {bh, r};
-                blas_op(c, OP_BMR_NORM, Pd, f, nullptr, &r2);  // r = bhat - r
-            }
-            flops += matpc_flops;
-            convert_op(c, rs, Ps, r, Pd);
-            rNorm = std::sqrt(r2);
-            maxrr = rNorm;
-            const bool restart = blown;
-            if (updX || restart) {
-                r0Norm = rNorm;
-                maxrx = rNorm;
-            }
-            SolverScalars upd = hs;
-            if (restart) {  // restart: rhat0 = r, p = r (beta = 0, v = 0)
-                copy(c, r0, rs, Ps);
-                zero(c, p, Ps);
-                zero(c, v, Ps);
-                const cd rn = cdot_of(c, Ps, r0, rs);
-                upd.rho = make_double2(1, 0);
-                upd.rho_new = make_double2(rn.real(), rn.imag());
-                upd.alpha = make_double2(1, 0);
-                upd.omega = make_double2(1, 0);
-                upd.beta = make_double2(0, 0);
-                ++restarts;
-            } else {
-                // continue the recurrences from the replaced residual: rho' = <rhat0, r>,
-                // beta = (rho'/rho)(alpha/omega) with the iteration's rho, alpha, omega
-                const cd rn = cdot_of(c, Ps, r0, rs);
-                const cd rho(hs.rho.x, hs.rho.y), al(hs.alpha.x, hs.alpha.y), om(hs.omega.x, hs.omega.y);
-                const cd beta = (rn / rho) * (al / om);
-                upd.rho_new = make_double2(rn.real(), rn.imag());
-                upd.beta = make_double2(beta.real(), beta.imag());
-            }
-            QX_CUDA(cudaMemcpyAsync(S, &upd, sizeof(upd), cudaMemcpyHostToDevice, c->stream));
-            QX_CUDA(cudaStreamSynchronize(c->stream));
-            ++updates;
-            if (rNorm <= stop) converged = true;
+        k = hs.k;
+        if (!hs.halt) continue;
+        // ---- reliable update requested by iteration k (Algorithm R; reading R3 for `blown`)
+        const double rNorm_it = hs.rNorm;
+        const bool blown = hs.blown != 0, updX = hs.updX != 0;
+        if (std::isfinite(rNorm_it)) xpy_mixed_op(c, Pd, Ps, xs, x_e);   // x += xs
+        zero(c, xs, Ps);
+        matpc_op(c, r, x_e, Pd, 0);          // r = Mhat x (high)
+        double r2;
+        {
+            void *f[2] = {bh, r};
+            blas_op(c, OP_BMR_NORM, Pd, f, nullptr, &r2);  // r = bhat - r
         }
+        flops += matpc_flops;
+        convert_op(c, rs, Ps, r, Pd);
+        const double rNorm = std::sqrt(r2);
+        SolverScalars upd = hs;
+        upd.halt = 0;
+        upd.updX = upd.blown = 0;
+        upd.rNorm = rNorm;
+        upd.maxrr = rNorm;
+        if (updX || blown) upd.r0Norm = upd.maxrx = rNorm;
+        if (blown) {  // restart: rhat0 = r, p = r (beta = 0, v = 0)
+            copy(c, r0, rs, Ps);
+            zero(c, p, Ps);
+            zero(c, v, Ps);
+            const cd rn = cdot_of(c, Ps, r0, rs);
+            upd.rho = make_double2(1, 0);
+            upd.rho_new = make_double2(rn.real(), rn.imag());
+            upd.alpha = make_double2(1, 0);
+            upd.omega = make_double2(1, 0);
+            upd.beta = make_double2(0, 0);
+            ++restarts;
+        } else {
+            // continue the recurrences from the replaced residual: rho' = <rhat0, r>,
+            // beta = (rho'/rho)(alpha/omega) with the iteration's rho, alpha, omega
+            const cd rn = cdot_of(c, Ps, r0, rs);
+            const cd rho(hs.rho.x, hs.rho.y), al(hs.alpha.x, hs.alpha.y), om(hs.omega.x, hs.omega.y);
+            const cd beta = (rn / rho) * (al / om);
+            upd.rho_new = make_double2(rn.real(), rn.imag());
+            upd.beta = make_double2(beta.real(), beta.imag());
+        }
+        *hS = upd;  // (the stream is idle: blas_op / cdot_of synchronised)
+        QX_CUDA(cudaMemcpyAsync(S, hS, sizeof(*hS), cudaMemcpyHostToDevice, c->stream));
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        ++updates;
         if (sp->res_history && k - 1 < sp->history_cap) sp->res_history[k - 1] = bnorm > 0 ? rNorm / bnorm : 0.0;
+        if (rNorm <= stop) converged = true;
+        st->true_res_schur = bnorm > 0 ? rNorm / bnorm : 0.0;
     }
-    if (gexec) cudaGraphExecDestroy(gexec);
-    release_graph_timing(c);
     st->iters = k;
     st->reliable_updates = updates;
     st->restarts = restarts;
-    st->true_res_schur = bnorm > 0 ? rNorm / bnorm : 0.0;
+    if (k == 0) st->true_res_schur = bnorm > 0 ? 1.0 : 0.0;
 
     finish_solution(c, Pd, x_dev, b_e, b_o, x_e, x_o, t_e, t_o, sp->use_schur, st);
     st->flops = flops;
@@ -377,11 +455,8 @@ void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_
     const double matpc_flops = mm.flops * V_h_all, blas_flops_iter = 960.0 * V_h_all;
     for (int j = 0; j < n; ++j) {
         auto &w = c->mws[j];
-        if (w.prec != Pd || w.prec_s != Ps) {
-            w = qudax_ctx::SolverWs{};
-            w.prec = Pd;
-            w.prec_s = Ps;
-        }
+        if (j == 0) QX_CUDA(cudaStreamSynchronize(c->stream));
+        ws_select(c, w, Pd, Ps);
         Sys &y = sys[j];
         y.b_e = field(c, w.b_e, Pd); y.b_o = field(c, w.b_o, Pd); y.bh = field(c, w.bh, Pd);
         y.x_e = field(c, w.x_e, Pd); y.x_o = field(c, w.x_o, Pd); y.r = field(c, w.r, Pd);
@@ -446,29 +521,30 @@ void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_
         }
         QX_CUDA(cudaMemcpyAsync(c->h_scal_m, c->d_scal_m, sizeof(SolverScalars) * n, cudaMemcpyDeviceToHost, c->stream));
     };
-    const bool use_graph = (c->comm != QUDAX_COMM_HOST) && !c->no_graphs && (c->g.nranks == 1 || c->force_graphs);
-    std::map<unsigned, std::pair<cudaGraphExec_t, long long>> graphs;  // one per active set
+    const bool use_graph = (c->comm != QUDAX_COMM_HOST) && !(c->flags & QUDAX_FLAG_NO_GRAPHS);
     bool first = true;
     for (;;) {
         unsigned mask = 0;
         for (int j = 0; j < n; ++j)
             if (sys[j].active) mask |= 1u << j;
         if (!mask) break;
+        const std::vector<qudax_ctx::TimingRec> *grecs = nullptr;
         if (!use_graph || first) {
             enqueue_iteration(mask);  // the first iteration runs eagerly (lazily-created buffers)
             first = false;
         } else {
-            auto it = graphs.find(mask);
-            if (it == graphs.end()) {
-                long long nl = 0;
-                cudaGraphExec_t e = capture_graph(c, [&] { enqueue_iteration(mask); }, &nl);
-                it = graphs.emplace(mask, std::make_pair(e, nl)).first;
-            }
-            QX_CUDA(cudaGraphLaunch(it->second.first, c->stream));
-            c->launches += it->second.second;
+            // one cached graph per active set (and workspace): every system's fields and scalars
+            std::vector<uintptr_t> key = {2, (uintptr_t)Pd, (uintptr_t)Ps, (uintptr_t)mask, (uintptr_t)n,
+                                          (uintptr_t)c->d_scal_m};
+            for (int j = 0; j < n; ++j)
+                for (void *f : {sys[j].rs, sys[j].xs, sys[j].p, sys[j].v, sys[j].t, sys[j].r0}) key.push_back((uintptr_t)f);
+            auto &gr = cached_graph(c, key, [&] { enqueue_iteration(mask); });
+            QX_CUDA(cudaGraphLaunch(gr.exec, c->stream));
+            c->launches += gr.launches;
+            grecs = &gr.trecs;
         }
         QX_CUDA(cudaStreamSynchronize(c->stream));
-        harvest_graph_timing(c);
+        if (grecs) harvest_graph_timing(c, *grecs, 1);
         for (int j = 0; j < n; ++j) {
             Sys &y = sys[j];
             if (!y.active) continue;
@@ -529,8 +605,6 @@ void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_
                 sp->res_history[y.k - 1] = y.bnorm > 0 ? y.rNorm / y.bnorm : 0.0;
         }
     }
-    for (auto &kv : graphs) cudaGraphExecDestroy(kv.second.first);
-    release_graph_timing(c);
     for (int j = 0; j < n; ++j) {
         Sys &y = sys[j];
         st[j].iters = y.k;
@@ -556,10 +630,8 @@ void cgnr_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_solv
     QX_CHECK(sp->maxiter >= 0 && sp->tol >= 0, QUDAX_ERR_ARG, "cgnr: bad parameters");
     std::memset(st, 0, sizeof(*st));
     auto &w = c->cgws;
-    if (w.prec != P) {
-        w = qudax_ctx::SolverWs{};
-        w.prec = P;
-    }
+    QX_CUDA(cudaStreamSynchronize(c->stream));
+    ws_select(c, w, P, P);
     const Geom &g = c->g;
     void *b_e = field(c, w.b_e, P), *b_o = field(c, w.b_o, P), *bh = field(c, w.bh, P);
     void *x_e = field(c, w.x_e, P), *x_o = field(c, w.x_o, P), *r = field(c, w.r, P);

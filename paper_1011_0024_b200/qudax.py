@@ -22,6 +22,8 @@ EVEN, ODD = 0, 1
 HOP, CLOVER_INV, CLOVER_XPAY, CLOVER_INV_XPAY = 0, 1, 2, 3
 COMM_NONE, COMM_NCCL, COMM_HOST = 0, 1, 2
 HALO_COMM, HALO_P2P = 0, 1
+# qudax_init_flag bits (include/qudax.h): test / comparison switches, 0 = defaults
+FLAG_NO_GRAPHS, FLAG_DEBUG_SOLVER, FLAG_FORCE_SS, FLAG_ONE_RHS_PER_THREAD, FLAG_TIMING_BREAKDOWN = 1, 2, 4, 8, 16
 PREC_NAMES = {"half": 2, "single": 4, "double": 8, "f16": 2, "f32": 4, "f64": 8}
 
 STATUS = {0: "QUDAX_OK", 1: "QUDAX_ERR_ARG", 2: "QUDAX_ERR_STATE", 3: "QUDAX_ERR_CUDA", 4: "QUDAX_ERR_NCCL",
@@ -48,7 +50,8 @@ class InitParam(ctypes.Structure):
                 ("nccl_id", ctypes.c_void_p), ("stream", ctypes.c_size_t),
                 ("dev_alloc", ALLOC_FN), ("dev_free", FREE_FN), ("alloc_user", ctypes.c_void_p),
                 ("host_exchange", EXCHANGE_FN), ("host_allreduce", ALLREDUCE_FN), ("comm_user", ctypes.c_void_p),
-                ("halo", ctypes.c_int), ("proc_grid", ctypes.c_int * 4), ("split_mask", ctypes.c_int)]
+                ("halo", ctypes.c_int), ("proc_grid", ctypes.c_int * 4), ("split_mask", ctypes.c_int),
+                ("flags", ctypes.c_int), ("copy_threads", ctypes.c_int)]
 
 
 class GaugeParam(ctypes.Structure):
@@ -60,7 +63,8 @@ class GaugeParam(ctypes.Structure):
 class SolveParam(ctypes.Structure):
     _fields_ = [("tol", ctypes.c_double), ("delta", ctypes.c_double), ("maxiter", ctypes.c_int),
                 ("prec_sloppy", ctypes.c_int), ("prec", ctypes.c_int), ("use_schur", ctypes.c_int),
-                ("res_history", ctypes.POINTER(ctypes.c_double)), ("history_cap", ctypes.c_int)]
+                ("res_history", ctypes.POINTER(ctypes.c_double)), ("history_cap", ctypes.c_int),
+                ("poll_every", ctypes.c_int)]
 
 
 class SolveStats(ctypes.Structure):
@@ -248,7 +252,8 @@ class Context:
     spinor_bytes(prec) bytes holding one parity in the library's layout."""
 
     def __init__(self, global_dims, nranks=1, rank=0, device=0, comm=COMM_NONE, overlap=True, nccl_id=None,
-                 stream=None, torch_allocator=True, transport=None, halo=HALO_COMM, proc_grid=None, split_mask=0):
+                 stream=None, torch_allocator=True, transport=None, halo=HALO_COMM, proc_grid=None, split_mask=0,
+                 flags=0, copy_threads=0):
         import torch
         self._torch = torch
         self.global_dims = tuple(int(d) for d in global_dims)
@@ -264,6 +269,7 @@ class Context:
         if proc_grid is not None:
             p.proc_grid = (ctypes.c_int * 4)(*proc_grid)
         p.split_mask = int(split_mask)
+        p.flags, p.copy_threads = int(flags), int(copy_threads)
         self._id = None
         if comm == COMM_NCCL:
             self._id = ctypes.create_string_buffer(bytes(nccl_id), 128)
@@ -297,6 +303,58 @@ class Context:
         self._check(lib().qudax_get_partition(self._h, ctypes.byref(part)))
         self.partition = part.as_dict()
         self.local_dims = tuple(self.partition["local_dims"])
+
+    # -- argument validation (every pointer handed to the library is checked first: a CUDA tensor
+    # given to a host entry point, a float32 or undersized buffer would otherwise be read or
+    # written out of bounds by the C side)
+    @property
+    def _slab_reals(self):
+        X, Y, Z, T_loc = self.local_dims
+        return 24 * X * Y * Z * T_loc
+
+    def _host_slab(self, a, name, writable=False):
+        """A full local slab in host memory: numpy complex128 [T_loc, Z, Y, X, 4, 3] or a CPU
+        float64 / complex128 torch tensor with the same number of reals; returns a double*."""
+        X, Y, Z, T_loc = self.local_dims
+        if hasattr(a, "data_ptr"):
+            torch = self._torch
+            if a.device.type != "cpu":
+                raise ValueError(f"{name}: host entry point needs a CPU tensor, got {a.device}")
+            if a.dtype not in (torch.float64, torch.complex128) or not a.is_contiguous():
+                raise ValueError(f"{name}: need a contiguous float64/complex128 tensor, got {a.dtype}")
+            reals = a.numel() * (2 if a.dtype == torch.complex128 else 1)
+            if reals != self._slab_reals:
+                raise ValueError(f"{name}: {reals} reals, the local slab has {self._slab_reals}")
+            return ctypes.cast(a.data_ptr(), _DP)
+        if not isinstance(a, np.ndarray) or a.dtype != np.complex128 or not a.flags.c_contiguous:
+            raise ValueError(f"{name}: need a C-contiguous complex128 numpy array")
+        if a.shape != (T_loc, Z, Y, X, 4, 3):
+            raise ValueError(f"{name}: shape {a.shape}, expected {(T_loc, Z, Y, X, 4, 3)}")
+        if writable and not a.flags.writeable:
+            raise ValueError(f"{name}: array is read-only")
+        return a.ctypes.data_as(_DP)
+
+    def _dev_slab(self, t, name):
+        """A full local slab on this context's GPU: contiguous float64 (or complex128) tensor."""
+        torch = self._torch
+        if not hasattr(t, "data_ptr") or t.device.type != "cuda" or t.device.index != self.device:
+            raise ValueError(f"{name}: need a CUDA tensor on cuda:{self.device}")
+        if t.dtype not in (torch.float64, torch.complex128) or not t.is_contiguous():
+            raise ValueError(f"{name}: need a contiguous float64/complex128 CUDA tensor, got {t.dtype}")
+        reals = t.numel() * (2 if t.dtype == torch.complex128 else 1)
+        if reals != self._slab_reals:
+            raise ValueError(f"{name}: {reals} reals, the local slab has {self._slab_reals}")
+        return t.data_ptr()
+
+    def _field(self, f, prec, name="field"):
+        """A parity field: a CUDA uint8 tensor of at least spinor_bytes(prec) bytes on this GPU."""
+        if f is None:
+            return None
+        if not hasattr(f, "data_ptr") or f.device.type != "cuda" or f.device.index != self.device:
+            raise ValueError(f"{name}: need a CUDA tensor on cuda:{self.device}")
+        if not f.is_contiguous() or f.numel() * f.element_size() < self.spinor_bytes(prec):
+            raise ValueError(f"{name}: need a contiguous buffer of >= {self.spinor_bytes(prec)} bytes")
+        return f.data_ptr()
 
     # -- plumbing
     def _check(self, st, ctx=True):
@@ -356,102 +414,117 @@ class Context:
         psi = np.ascontiguousarray(psi, dtype=np.complex128)
         X, Y, Z, T_loc = self.local_dims
         assert psi.shape == (T_loc, Z, Y, X, 4, 3), psi.shape
-        self._check(lib().qudax_spinor_load(self._h, field.data_ptr(), int(prec), int(parity), _dptr(psi)))
+        self._check(lib().qudax_spinor_load(self._h, self._field(field, prec), int(prec), int(parity), _dptr(psi)))
 
     def spinor_load_dev(self, field, prec, parity, src):
-        self._check(lib().qudax_spinor_load_dev(self._h, field.data_ptr(), int(prec), int(parity), src.data_ptr()))
+        self._check(lib().qudax_spinor_load_dev(self._h, self._field(field, prec), int(prec), int(parity),
+                                                self._dev_slab(src, "src")))
 
     def spinor_store(self, field, prec, parity, out=None):
         X, Y, Z, T_loc = self.local_dims
         if out is None:
             out = np.zeros((T_loc, Z, Y, X, 4, 3), dtype=np.complex128)
-        self._check(lib().qudax_spinor_store(self._h, _dptr(out), field.data_ptr(), int(prec), int(parity)))
+        op = self._host_slab(out, "out", writable=True)
+        self._check(lib().qudax_spinor_store(self._h, op, self._field(field, prec), int(prec), int(parity)))
         return out
 
     def spinor_store_dev(self, dst, field, prec, parity):
-        self._check(lib().qudax_spinor_store_dev(self._h, dst.data_ptr(), field.data_ptr(), int(prec), int(parity)))
+        self._check(lib().qudax_spinor_store_dev(self._h, self._dev_slab(dst, "dst"), self._field(field, prec), int(prec),
+                                                 int(parity)))
 
     def convert(self, dst, dst_prec, src, src_prec):
-        self._check(lib().qudax_spinor_convert(self._h, dst.data_ptr(), int(dst_prec), src.data_ptr(), int(src_prec)))
+        self._check(lib().qudax_spinor_convert(self._h, self._field(dst, dst_prec, "dst"), int(dst_prec),
+                                               self._field(src, src_prec, "src"), int(src_prec)))
 
     # -- operator
     def dslash(self, out, inp, prec, out_parity, dagger=False, kind=HOP, x=None, a=0.0):
-        xp = x.data_ptr() if x is not None else None
-        self._check(lib().qudax_dslash(self._h, out.data_ptr(), inp.data_ptr(), xp, int(prec), int(out_parity),
+        xp = self._field(x, prec, "x")
+        self._check(lib().qudax_dslash(self._h, self._field(out, prec, "out"), self._field(inp, prec, "in"), xp,
+                                       int(prec), int(out_parity),
                                        int(bool(dagger)), int(kind), float(a)))
 
     def matpc(self, out, inp, prec, dagger=False):
-        self._check(lib().qudax_matpc(self._h, out.data_ptr(), inp.data_ptr(), int(prec), int(bool(dagger))))
+        self._check(lib().qudax_matpc(self._h, self._field(out, prec, "out"), self._field(inp, prec, "in"), int(prec),
+                                      int(bool(dagger))))
 
     def matpc_sym(self, out, inp, prec, dagger=False):
         """Symmetric Schur form T_ee^{-1} Mhat (or its explicit adjoint)."""
-        self._check(lib().qudax_matpc_sym(self._h, out.data_ptr(), inp.data_ptr(), int(prec), int(bool(dagger))))
+        self._check(lib().qudax_matpc_sym(self._h, self._field(out, prec, "out"), self._field(inp, prec, "in"),
+                                          int(prec), int(bool(dagger))))
 
-    @staticmethod
-    def _ptrs(fields):
-        return (_P * len(fields))(*[f.data_ptr() for f in fields])
+    def _ptrs(self, fields, prec):
+        return (_P * len(fields))(*[self._field(f, prec) for f in fields])
 
     def dslash_multi(self, outs, ins, prec, out_parity, dagger=False, kind=HOP, xs=None, a=0.0):
-        xp = self._ptrs(xs) if xs is not None else None
-        self._check(lib().qudax_dslash_multi(self._h, self._ptrs(outs), self._ptrs(ins), xp, len(ins), int(prec),
+        if len(outs) != len(ins) or (xs is not None and len(xs) != len(ins)):
+            raise ValueError("dslash_multi: outs / ins / xs lengths differ")
+        xp = self._ptrs(xs, prec) if xs is not None else None
+        self._check(lib().qudax_dslash_multi(self._h, self._ptrs(outs, prec), self._ptrs(ins, prec), xp, len(ins), int(prec),
                                              int(out_parity), int(bool(dagger)), int(kind), float(a)))
 
     def matpc_multi(self, outs, ins, prec, dagger=False):
-        self._check(lib().qudax_matpc_multi(self._h, self._ptrs(outs), self._ptrs(ins), len(ins), int(prec),
+        if len(outs) != len(ins):
+            raise ValueError("matpc_multi: outs / ins lengths differ")
+        self._check(lib().qudax_matpc_multi(self._h, self._ptrs(outs, prec), self._ptrs(ins, prec), len(ins), int(prec),
                                             int(bool(dagger))))
 
     def mdagm(self, out, inp, prec):
-        self._check(lib().qudax_mdagm(self._h, out.data_ptr(), inp.data_ptr(), int(prec)))
+        self._check(lib().qudax_mdagm(self._h, self._field(out, prec, "out"), self._field(inp, prec, "in"), int(prec)))
 
     def norm2(self, f, prec):
         r = ctypes.c_double()
-        self._check(lib().qudax_norm2(self._h, f.data_ptr(), int(prec), ctypes.byref(r)))
+        self._check(lib().qudax_norm2(self._h, self._field(f, prec), int(prec), ctypes.byref(r)))
         return r.value
 
     def cdot(self, a, b, prec):
         r = (ctypes.c_double * 2)()
-        self._check(lib().qudax_cdot(self._h, a.data_ptr(), b.data_ptr(), int(prec), r))
+        self._check(lib().qudax_cdot(self._h, self._field(a, prec, "a"), self._field(b, prec, "b"), int(prec), r))
         return complex(r[0], r[1])
 
     # -- solver
-    def _solve_param(self, tol, delta, maxiter, prec, prec_sloppy, use_schur, history=None):
+    def _solve_param(self, tol, delta, maxiter, prec, prec_sloppy, use_schur, history=None, poll_every=0):
         # use_schur: True/1 asymmetric Schur form, 2 (or "sym") symmetric, False/0 even system only
         us = 2 if use_schur in (2, "sym") else int(bool(use_schur))
         sp = SolveParam(float(tol), float(delta), int(maxiter), int(prec_sloppy), int(prec), us)
         if history is not None:
-            assert history.dtype == np.float64 and history.flags.c_contiguous
+            if not isinstance(history, np.ndarray) or history.dtype != np.float64 or not history.flags.c_contiguous:
+                raise ValueError("history: need a C-contiguous float64 numpy array")
             sp.res_history = history.ctypes.data_as(_DP)
             sp.history_cap = int(history.size)
+        sp.poll_every = int(poll_every)
         return sp
+
+    def _finish(self, rc, allow_not_converged):
+        if rc and not (allow_not_converged and rc == 6):
+            self._check(rc)
 
     def solve_cgnr(self, b, tol=1e-10, maxiter=10000, prec=DOUBLE, use_schur=True, allow_not_converged=False,
                    history=None):
         """CGNR on Mhat^dag Mhat in one precision; host arrays as in solve()."""
         b = np.ascontiguousarray(b, dtype=np.complex128)
         x = np.zeros_like(b)
+        bp, xp = self._host_slab(b, "b"), self._host_slab(x, "x", writable=True)
         sp = self._solve_param(tol, 0.0, maxiter, prec, prec, use_schur, history)
         st = SolveStats()
-        rc = lib().qudax_solve_cgnr(self._h, _dptr(x), _dptr(b), ctypes.byref(sp), ctypes.byref(st))
-        if rc and not (allow_not_converged and rc == 6):
-            self._check(rc)
+        self._finish(lib().qudax_solve_cgnr(self._h, xp, bp, ctypes.byref(sp), ctypes.byref(st)), allow_not_converged)
         return x, st.as_dict()
 
     def solve(self, b, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
-              allow_not_converged=False, history=None, out=None):
+              allow_not_converged=False, history=None, out=None, poll_every=0):
         """x = M^{-1} b (host arrays, full local slab, DR basis); returns (x, stats dict).
-        history: optional float64 numpy array receiving ||r_k||/||bhat|| per iteration."""
-        if hasattr(b, "data_ptr"):  # torch CPU tensors (e.g. pinned float64 buffers), x preallocated
-            bp, x = ctypes.cast(b.data_ptr(), _DP), (out if out is not None else self._torch.zeros_like(b))
-            xp = ctypes.cast(x.data_ptr(), _DP)
+        b: numpy complex128 [T_loc, Z, Y, X, 4, 3] or a CPU float64 torch tensor of the same size
+        (e.g. a pinned buffer; then `out` may be a preallocated one).  history: optional float64
+        numpy array receiving ||r_k||/||bhat|| per iteration."""
+        if hasattr(b, "data_ptr"):
+            x = out if out is not None else self._torch.zeros_like(b)
         else:
             b = np.ascontiguousarray(b, dtype=np.complex128)
             x = np.zeros_like(b) if out is None else out
-            bp, xp = _dptr(b), _dptr(x)
-        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history)
+        bp, xp = self._host_slab(b, "b"), self._host_slab(x, "out", writable=True)
+        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history, poll_every)
         st = SolveStats()
-        rc = lib().qudax_solve_bicgstab(self._h, xp, bp, ctypes.byref(sp), ctypes.byref(st))
-        if rc and not (allow_not_converged and rc == 6):
-            self._check(rc)
+        self._finish(lib().qudax_solve_bicgstab(self._h, xp, bp, ctypes.byref(sp), ctypes.byref(st)),
+                     allow_not_converged)
         return x, st.as_dict()
 
     def solve_multi(self, bs, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
@@ -460,36 +533,46 @@ class Context:
         Mhat kernel pair per iteration for all still-active systems.  Returns (xs, [stats])."""
         bs = [np.ascontiguousarray(b, dtype=np.complex128) for b in bs]
         xs = outs if outs is not None else [np.zeros_like(b) for b in bs]
+        if len(xs) != len(bs):
+            raise ValueError("solve_multi: outs / bs lengths differ")
         n = len(bs)
-        bp = (_P * n)(*[b.ctypes.data for b in bs])
-        xp = (_P * n)(*[x.ctypes.data for x in xs])
+        bp = (_P * n)(*[ctypes.cast(self._host_slab(b, f"bs[{j}]"), _P).value for j, b in enumerate(bs)])
+        xp = (_P * n)(*[ctypes.cast(self._host_slab(x, f"outs[{j}]", writable=True), _P).value for j, x in enumerate(xs)])
         sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history)
         st = (SolveStats * n)()
-        rc = lib().qudax_solve_bicgstab_multi(self._h, xp, bp, n, ctypes.byref(sp), st)
-        if rc and not (allow_not_converged and rc == 6):
-            self._check(rc)
+        self._finish(lib().qudax_solve_bicgstab_multi(self._h, xp, bp, n, ctypes.byref(sp), st), allow_not_converged)
         return xs, [s.as_dict() for s in st]
 
     def solve_multi_dev(self, xs, bs, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE,
                         use_schur=True, allow_not_converged=False):
         """Device-resident batched solve: lists of float64 CUDA tensors (full local slabs)."""
+        if len(xs) != len(bs):
+            raise ValueError("solve_multi_dev: xs / bs lengths differ")
         n = len(bs)
-        bp = (_P * n)(*[b.data_ptr() for b in bs])
-        xp = (_P * n)(*[x.data_ptr() for x in xs])
+        bp = (_P * n)(*[self._dev_slab(b, f"bs[{j}]") for j, b in enumerate(bs)])
+        xp = (_P * n)(*[self._dev_slab(x, f"xs[{j}]") for j, x in enumerate(xs)])
         sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur)
         st = (SolveStats * n)()
-        rc = lib().qudax_solve_bicgstab_multi_dev(self._h, xp, bp, n, ctypes.byref(sp), st)
-        if rc and not (allow_not_converged and rc == 6):
-            self._check(rc)
+        self._finish(lib().qudax_solve_bicgstab_multi_dev(self._h, xp, bp, n, ctypes.byref(sp), st),
+                     allow_not_converged)
         return [s.as_dict() for s in st]
 
     def solve_dev(self, x, b, tol=1e-10, delta=0.1, maxiter=10000, prec=DOUBLE, prec_sloppy=SINGLE, use_schur=True,
-                  allow_not_converged=False, history=None):
+                  allow_not_converged=False, history=None, poll_every=0):
         """Device-resident variant: x, b are float64 CUDA tensors holding the full local slab
         (T_loc, Z, Y, X, 4, 3, 2)."""
-        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history)
+        xp, bp = self._dev_slab(x, "x"), self._dev_slab(b, "b")
+        sp = self._solve_param(tol, delta, maxiter, prec, prec_sloppy, use_schur, history, poll_every)
         st = SolveStats()
-        rc = lib().qudax_solve_bicgstab_dev(self._h, x.data_ptr(), b.data_ptr(), ctypes.byref(sp), ctypes.byref(st))
-        if rc and not (allow_not_converged and rc == 6):
-            self._check(rc)
+        self._finish(lib().qudax_solve_bicgstab_dev(self._h, xp, bp, ctypes.byref(sp), ctypes.byref(st)),
+                     allow_not_converged)
+        return st.as_dict()
+
+    def solve_cgnr_dev(self, x, b, tol=1e-10, maxiter=10000, prec=DOUBLE, use_schur=True, allow_not_converged=False):
+        """Device-resident CGNR (x, b as in solve_dev)."""
+        xp, bp = self._dev_slab(x, "x"), self._dev_slab(b, "b")
+        sp = self._solve_param(tol, 0.0, maxiter, prec, prec, use_schur)
+        st = SolveStats()
+        self._finish(lib().qudax_solve_cgnr_dev(self._h, xp, bp, ctypes.byref(sp), ctypes.byref(st)),
+                     allow_not_converged)
         return st.as_dict()

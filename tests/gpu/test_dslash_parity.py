@@ -46,6 +46,10 @@ def get_case(name):
             _cases[name] = Case((8, 4, 6, 8), 1011, 2011)
         elif name == "16^3x32":
             _cases[name] = Case((16, 16, 16, 32), 1002, 2002)
+        elif name == "8x4x6x8 periodic":
+            _cases[name] = Case((8, 4, 6, 8), 1011, 2011, t_bc=+1)
+        elif name == "16^3x32 periodic":
+            _cases[name] = Case((16, 16, 16, 32), 1002, 2002, t_bc=+1)
     return _cases[name]
 
 
@@ -97,6 +101,37 @@ def test_dslash_small_lattices(torch_cuda, name, prec):
         ctx.close()
 
 
+@pytest.mark.parametrize("prec", [8, 4, 2])
+@pytest.mark.parametrize("recon", [18, 12, 8])
+def test_dslash_periodic_t(torch_cuda, prec, recon):
+    """t_boundary = +1 (periodic in T; P:381-383 and P:625-628 leave the boundary constants to
+    the caller, reading Q5): every precision, reconstruct, parity, dagger and kind at 16^3x32,
+    Mhat and Mhat^dag at 8x4x6x8.  With recon 12 the third row is rebuilt BEFORE the sign, so an
+    in-storage sign flip would fail here and in the antiperiodic matrix alike."""
+    case = get_case("16^3x32 periodic")
+    ctx = make_ctx(case, prec, recon)
+    for p in (0, 1):
+        for dagger in (False, True):
+            for kind in (qudax.HOP, qudax.CLOVER_INV, qudax.CLOVER_XPAY):
+                got = run_dslash(ctx, case, prec, p, dagger, kind, -0.37)
+                e = rel_l2(got, case.expect(p, dagger, kind, -0.37))
+                assert e <= TOL[prec], (prec, recon, p, dagger, kind, e)
+    ctx.close()
+    small = get_case("8x4x6x8 periodic")
+    ctx = make_ctx(small, prec, recon)
+    psi_e = oracle.restrict(small.psi, 0)
+    fin, fout = ctx.new_field(prec), ctx.new_field(prec)
+    ctx.spinor_load(fin, prec, 0, small.psi)
+    for dagger in (False, True):
+        ctx.matpc(fout, fin, prec, dagger)
+        got = oracle.restrict(ctx.spinor_store(fout, prec, 0), 0)
+        assert rel_l2(got, small.wc.matpc(psi_e, dagger)) <= TOL[prec], dagger
+    # the periodic and antiperiodic operators must differ (the sign is not silently dropped)
+    anti = oracle.WilsonClover(small.U, small.kappa, small.csw, -1).matpc(psi_e)
+    assert rel_l2(got, anti) > 0.05  # measured 0.11 in fp64 on this lattice
+    ctx.close()
+
+
 def test_wilson_csw0_4x4(torch_cuda):
     case = Case((4, 4, 4, 4), 1001, 2001, kappa=0.12, csw=0.0)
     ctx = make_ctx(case, 8, 18)
@@ -119,7 +154,7 @@ def test_matpc_and_mdagm(torch_cuda, prec, recon):
         assert rel_l2(got, case.wc.matpc(psi_e, dagger)) <= TOL[prec]
     ctx.mdagm(fout, fin, prec)
     got = oracle.restrict(ctx.spinor_store(fout, prec, 0), 0)
-    assert rel_l2(got, case.wc.mdagm(psi_e)) <= TOL[prec] * (3 if prec == 2 else 1)
+    assert rel_l2(got, case.wc.mdagm(psi_e)) <= TOL[prec]
     ctx.close()
 
 

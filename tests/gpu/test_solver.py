@@ -246,3 +246,78 @@ def test_batched_equals_independent_at_config3_size(torch_cuda):
         assert (st["iters"], st["reliable_updates"]) == (one["iters"], one["reliable_updates"])
         assert st["true_res"] <= 1e-14 * (1 + 1e-3)
     ctx.close()
+
+
+def test_poll_every_and_eager_are_bitwise_identical(torch_cuda, system):
+    """Algorithm R's update rule runs on the device after every iteration; the host reads the
+    scalars once per batch of poll_every iterations (one CUDA-graph replay), and an iteration that
+    asks for a reliable update voids the rest of its batch.  The iterates must therefore not
+    depend on the batch size or on graph replay: bitwise equal x, the same iteration count,
+    updates and residual history for poll_every 1 / 3 / 4 / 16 and with graphs disabled."""
+    U, wc = system
+    b = qgen.point_source(DIMS, 0, 1)
+    runs = []
+    for flags, poll in ((0, 1), (0, 3), (0, 4), (0, 16), (qudax.FLAG_NO_GRAPHS, 4)):
+        ctx = qudax.Context(DIMS, flags=flags)
+        ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+        h = np.zeros(400)
+        x, st = ctx.solve(b, tol=1e-12, delta=1e-2, maxiter=400, prec=8, prec_sloppy=4, history=h, poll_every=poll)
+        runs.append((x, st, h))
+        ctx.close()
+    x0, st0, h0 = runs[0]
+    assert st0["reliable_updates"] >= 2
+    for x, st, h in runs[1:]:
+        assert st["iters"] == st0["iters"] and st["reliable_updates"] == st0["reliable_updates"]
+        assert np.array_equal(x, x0)
+        assert np.array_equal(h, h0)
+    res = np.linalg.norm(wc.M(x0) - b) / np.linalg.norm(b)
+    assert res <= 1e-12 * (1 + 1e-3)
+
+
+def test_loopback_nccl_solve_bitwise_with_allreduce_in_graph(torch_cuda, system):
+    """The N > 1 code path on one GPU: NCCL loopback without overlap (pack -> ncclSend/Recv to
+    self -> one whole-lattice kernel, so the fused reductions keep the unsplit CTA grouping), the
+    three per-iteration sums through ncclAllReduce on the one-rank communicator followed by the
+    coefficient kernel, all captured in the cached iteration graph.  Must be bitwise equal to the
+    unsplit solve (the exchange and the one-rank allreduce move bits only)."""
+    U, wc = system
+    b = qgen.point_source(DIMS, 1, 1)
+    out = []
+    for comm in (qudax.COMM_NONE, qudax.COMM_NCCL):
+        ctx = qudax.Context(DIMS, comm=comm, overlap=False, nccl_id=qudax.nccl_unique_id() if comm else None)
+        ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+        h = np.zeros(400)
+        for _ in range(2):  # the second solve replays the cached graph
+            x, st = ctx.solve(b, tol=1e-11, delta=1e-2, maxiter=400, prec=8, prec_sloppy=4, history=h)
+        out.append((x, st, h.copy()))
+        ctx.close()
+    assert out[0][1]["iters"] == out[1][1]["iters"]
+    assert np.array_equal(out[0][2], out[1][2])
+    assert np.array_equal(out[0][0], out[1][0])
+
+
+def test_binding_rejects_bad_buffers(torch_cuda, system):
+    """The binding validates every pointer it hands to the library: a CUDA tensor
+    on a host entry point, float32 or undersized buffers, a host array on a device entry point."""
+    import torch
+    U, _ = system
+    ctx = qudax.Context(DIMS)
+    ctx.gauge_load(U, KAPPA, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+    b = qgen.point_source(DIMS, 0, 0)
+    bd = torch.from_numpy(b.view(np.float64).copy()).cuda()
+    with pytest.raises(ValueError):
+        ctx.solve(bd)                                   # device tensor to the host entry
+    with pytest.raises(ValueError):
+        ctx.solve(b, out=np.zeros(10, dtype=np.complex128))
+    with pytest.raises(ValueError):
+        ctx.solve_dev(torch.zeros_like(bd).float(), bd)  # float32 x
+    with pytest.raises(ValueError):
+        ctx.solve_dev(torch.zeros(100, dtype=torch.float64, device="cuda"), bd)
+    with pytest.raises(ValueError):
+        ctx.solve_dev(torch.zeros_like(bd).cpu(), bd)
+    f = ctx.new_field(4)
+    with pytest.raises(ValueError):
+        ctx.matpc(f, f[:100], 4)
+    with pytest.raises(ValueError):
+        ctx.matpc(ctx.new_field(2), ctx.new_field(2), 4)  # half-sized buffers for an fp32 operator
+    ctx.close()

@@ -40,6 +40,18 @@ def test_gamma4_projectors_match_eq6():
     assert np.allclose(S @ (np.eye(4) - g4) @ S.T, np.array(sec["P-4 nonrel"]), atol=1e-15)
 
 
+def test_gammas_match_appendix_a_golden():
+    """gamma_1..gamma_4 and gamma_5 entry by entry against the transcription of SURVEY.md
+    Appendix A (tests/golden/gamma_degrand_rossi.txt; gamma_4 also fixed by eq. (6)).
+    Clifford algebra alone admits any unitary rotation of the basis; this pins the one the API
+    documents (a swapped or sign-flipped gamma_mu changes which spin components a hop mixes)."""
+    sec, _ = read_golden("gamma_degrand_rossi.txt")
+    for mu in range(4):
+        want = np.array(sec[f"g{mu + 1} re"]) + 1j * np.array(sec[f"g{mu + 1} im"])
+        assert np.array_equal(oracle.gamma(mu), want), mu
+    assert np.array_equal(oracle.gamma5(), np.array(sec["g5 re"]))
+
+
 # --------------------------------------------------------------------------- generators
 
 def test_generator_su3_and_slab_independence():
@@ -414,3 +426,28 @@ def test_sampled_evaluation_matches_full():
     got = oracle.matpc_sites(U, psi_e, ev, 0.12, 1.1, -1.0)
     want = wc.matpc(psi_e).reshape(-1, 4, 3)[ev]
     assert np.abs(got - want).max() < 1e-13
+
+
+@pytest.mark.parametrize("chunk", [7, 13, 1 << 17])
+def test_apply_M_chunked_pins(chunk):
+    """oracle.apply_M_chunked (the full-size residual checker, T evaluated chunk by chunk with
+    clover_sites) against (i) the closed form on the unit gauge, where T = 1 and M_kappa =
+    1 - kappa D acts on a plane wave as e^{ip.x}(1 - kappa sum_mu (2 cos p_mu - 2 i gamma_mu
+    sin p_mu)) u (reading Q4; no oracle involved), and (ii) T - kappa D from the
+    whole-lattice clover (WilsonClover.M, pinned above by the abelian closed form and the dense
+    Schur complement) at odd chunk sizes that cut the lattice mid-timeslice.  Catches a dropped
+    chunk tail, a wrong -kappa sign, or the clover applied to the wrong sites."""
+    dims = (4, 4, 2, 6)
+    kappa, csw = 0.124, 1.0
+    u = RNG.normal(size=(4, 3)) + 1j * RNG.normal(size=(4, 3))
+    for antiperiodic in (True, False):
+        p, pw = _plane_wave(dims, (1, 1, 0, 2), antiperiodic, u)
+        Dt = sum(2 * np.cos(p[m]) * np.eye(4) - 2j * np.sin(p[m]) * oracle.gamma(m) for m in range(4))
+        expect = np.einsum("st,...tc->...sc", np.eye(4) - kappa * Dt, pw)
+        got = oracle.apply_M_chunked(qgen.unit_gauge(dims), pw, kappa, csw, -1.0 if antiperiodic else 1.0, chunk=chunk)
+        assert np.abs(got - expect).max() < 1e-13
+    U = qgen.gauge(dims, 93)
+    x = qgen.spinor(dims, 94)
+    wc = oracle.WilsonClover(U, kappa, csw, -1.0)
+    got = oracle.apply_M_chunked(U, x, kappa, csw, -1.0, chunk=chunk)
+    assert np.abs(got - wc.M(x)).max() < 1e-13 * np.abs(wc.M(x)).max()
