@@ -59,6 +59,7 @@ def parse():
     ap.add_argument("--scaling", default="weak", choices=["weak", "strong"],
                     help="weak: 32^3x64 per GPU (BASELINE configs[4]); strong: 32^3x256 in total (configs[3])")
     ap.add_argument("--oracle-sample", type=int, default=0, help=argparse.SUPPRESS)  # internal: 1-thread oracle run
+    ap.add_argument("--oracle-ops", action="store_true", help=argparse.SUPPRESS)  # internal: 1-thread oracle ops
     return ap.parse_args()
 
 
@@ -210,6 +211,89 @@ def single_gpu_extras(ctx, b_dev, peak):
     return out
 
 
+def oracle_operator_seconds(reps=1):
+    """SURVEY 8(d) timing protocol: the fp64 oracle's seconds per Dslash (eq. 2, all sites) and
+    per Mhat (even sites), on the box's host cores, for BASELINE configs[0..2] (4^4, 16^3x32,
+    24^3x128).  Returns {config: {"dslash_s", "matpc_s", "threads"}}; run once with the default
+    OpenMP thread count and once in a child with OMP_NUM_THREADS=1 (oracle_operator_seconds_1thread)."""
+    import numpy as np
+
+    import oracle
+    import qgen
+    out = {}
+    oracle.dslash(qgen.gauge((4, 4, 4, 4), 1), qgen.spinor((4, 4, 4, 4), 2))  # OpenMP thread start-up
+    for name, dims, gseed in (("configs[0] 4^4", (4, 4, 4, 4), 1001), ("configs[1] 16^3x32", (16, 16, 16, 32), 1002),
+                              ("configs[2] 24^3x128", (24, 24, 24, 128), 1003)):
+        U = qgen.gauge(dims, gseed, eps=-1.0 if gseed != 1003 else EPS)
+        psi = qgen.spinor(dims, gseed + 1000)
+        t0 = time.perf_counter()
+        for _ in range(reps):
+            oracle.dslash(U, psi, -1.0)
+        t_d = (time.perf_counter() - t0) / reps
+        wc = oracle.WilsonClover(U, KAPPA, CSW, -1.0)
+        pe = oracle.restrict(psi, 0)
+        t0 = time.perf_counter()
+        for _ in range(reps):
+            wc.matpc(pe)
+        t_m = (time.perf_counter() - t0) / reps
+        vh = np.prod(dims) / 2
+        out[name] = {"dslash_s": t_d, "matpc_s": t_m, "dslash_gflops": 1320 * 2 * vh / t_d * 1e-9,
+                     "matpc_gflops": 3696 * vh / t_m * 1e-9}
+        del U, psi, wc, pe
+    threads = int(os.environ.get("OMP_NUM_THREADS", os.cpu_count() or 1))
+    return {"threads": threads, "configs": out,
+            "note": "oracle = plain fp64 C (OpenMP) + numpy; Dslash over every site of the lattice, Mhat on the even "
+                    "sites (clover build excluded, done once per WilsonClover)"}
+
+
+def oracle_operator_seconds_1thread():
+    env = dict(os.environ, OMP_NUM_THREADS="1")
+    r = subprocess.run([sys.executable, os.path.abspath(__file__), "--oracle-ops"], env=env, capture_output=True,
+                       text=True, timeout=900)
+    if r.returncode != 0:
+        return None
+    return json.loads(r.stdout.strip().splitlines()[-1])
+
+
+def config2_l2_resident(peak):
+    """BASELINE configs[1]: 16^3x32 (fp32-12, 57 MB working set < the 126 MB L2): Mhat timed
+    back to back — the number is L2-RESIDENT, labelled so, not an HBM measurement."""
+    import torch
+
+    import qgen
+    from paper_1011_0024_b200 import qudax
+    dims = (16, 16, 16, 32)
+    ctx = qudax.Context(dims)
+    ctx.gauge_load(qgen.gauge(dims, 1002), 0.12, 1.0, prec=4, recon=12)
+    fi, fo = ctx.new_field(4), ctx.new_field(4)
+    ctx.spinor_load(fi, 4, 0, qgen.spinor(dims, 2002))
+    times = timed_reps(ctx, lambda: ctx.matpc(fo, fi, 4), 60)
+    ctx.close()
+    m = qudax.site_model(4, 12, -1)
+    vh = 16 ** 3 * 32 // 2
+    med = statistics.median(times)
+    return {"lattice": "16^3x32 fp32-12 Mhat", "l2_resident": True, "matpc_us_median": 1e3 * med,
+            "matpc_us_min": 1e3 * min(times), "reps": len(times),
+            "matpc_gflops_median": m["flops"] * vh / (med * 1e-3) * 1e-9,
+            "model_gbs_median": m["bytes_compulsory"] * vh / (med * 1e-3) * 1e-9,
+            "note": "working set ~57 MB < 126 MB L2: L2-resident bandwidth, not HBM"}
+
+
+def timed_reps(ctx, fn, reps, warm=5):
+    """Per-application times (ms) of `fn` on the context's stream: CUDA events around each of
+    `reps` back-to-back applications after `warm` untimed ones (SURVEY 8(d) timing protocol)."""
+    import torch
+    for _ in range(warm):
+        fn()
+    ev = [torch.cuda.Event(enable_timing=True) for _ in range(reps + 1)]
+    ev[0].record(ctx.stream)
+    for k in range(reps):
+        fn()
+        ev[k + 1].record(ctx.stream)
+    ctx.stream.synchronize()
+    return [ev[k].elapsed_time(ev[k + 1]) for k in range(reps)]
+
+
 def config3_solve_time():
     """BASELINE configs[2]: 24^3 x 128 weak field, the paper's 6 point sources (colour 0-2 x
     spin 0-1, P:748-751), mixed double-single (delta 1e-3, the paper's single-precision value;
@@ -282,6 +366,9 @@ def run_reference(args):
 
 # ---------------------------------------------------------------------------- our arm
 def main():
+    if "--oracle-ops" in sys.argv:  # child of oracle_operator_seconds_1thread (no GPU work)
+        print(json.dumps(oracle_operator_seconds()))
+        return
     if "--oracle-sample" in sys.argv:  # child of cpu_oracle_1thread (no GPU work)
         a = parse()
         g, dt, threads, sample = cpu_oracle_gflops(a.oracle_sample)
@@ -331,6 +418,8 @@ def main():
     if world > 1:
         obj = [qudax.nccl_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(obj, src=0)
+        obj2 = [qudax.nccl_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(obj2, src=0)
         ctx = qudax.Context(dims, nranks=N, rank=rank, device=local, comm=qudax.COMM_NCCL, nccl_id=obj[0],
                             overlap=bool(args.overlap), proc_grid=grid,
                             halo=qudax.HALO_P2P if args.halo == "p2p" else qudax.HALO_COMM)
@@ -412,40 +501,63 @@ def main():
 
     # ---- Dslash-only numbers (Mhat applications, device resident), per precision
     dslash = {}
+    vh_loc = local_dims[0] * local_dims[1] * local_dims[2] * T_loc // 2
+
+    def matpc_numbers(c, prec, recon, reps=50):
+        """Mhat applied `reps` times back to back: per-application CUDA-event times (median and
+        minimum, max over ranks of each), plus the Dslash kernels' own event times."""
+        fin, fout = c.new_field(prec), c.new_field(prec)
+        c.spinor_load_dev(fin, prec, 0, b_dev)
+        barrier()
+        c.kernel_timing(True)
+        times = timed_reps(c, lambda: c.matpc(fout, fin, prec), reps)
+        k2 = c.kernel_stats(prec=prec)
+        c.kernel_timing(False)
+        barrier()
+        med, mn = max_over_ranks(statistics.median(times)), max_over_ranks(min(times))
+        m = qudax.site_model(prec, recon, -1)
+        kg = k2["bytes_compulsory"] / (k2["ms_total"] * 1e-3) * 1e-9
+        return {"matpc_us_median": 1e3 * med, "matpc_us_min": 1e3 * mn, "reps": reps,
+                "matpc_gflops_total": m["flops"] * vh_loc * N / (med * 1e-3) * 1e-9,
+                "matpc_gflops_per_gpu": m["flops"] * vh_loc / (med * 1e-3) * 1e-9,
+                "model_gbs_per_gpu": m["bytes_compulsory"] * vh_loc / (med * 1e-3) * 1e-9,
+                "kernel_gbs_compulsory": kg, "kernel_gflops": k2["flops"] / (k2["ms_total"] * 1e-3) * 1e-9,
+                "frac_of_measured_hbm": kg / peak}
+
     if not args.no_extra:
         for prec, recon, name in ((4, 12, "fp32-12"), (8, 18, "fp64-18")):
-            fin, fout = ctx.new_field(prec), ctx.new_field(prec)
-            ctx.spinor_load_dev(fin, prec, 0, b_dev)
-            for _ in range(5):
-                ctx.matpc(fout, fin, prec)
-            barrier()
-            ctx.kernel_timing(True)
-            ea, eb = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-            reps = 50
-            ea.record(ctx.stream)
-            for _ in range(reps):
-                ctx.matpc(fout, fin, prec)
-            eb.record(ctx.stream)
-            barrier()
-            mms = max_over_ranks(ea.elapsed_time(eb))
-            k2 = ctx.kernel_stats(prec=prec)
-            ctx.kernel_timing(False)
-            m = qudax.site_model(prec, recon, -1)
-            sites = (local_dims[0] * local_dims[1] * local_dims[2] * T_loc // 2) * N
-            per_gpu = sites / N * reps
-            dslash[name] = {
-                "matpc_gflops_total": m["flops"] * sites * reps / (mms * 1e-3) * 1e-9,
-                "matpc_gflops_per_gpu": m["flops"] * per_gpu / (mms * 1e-3) * 1e-9,
-                "matpc_us": 1e3 * mms / reps,
-                "model_gbs_per_gpu": m["bytes_compulsory"] * per_gpu / (mms * 1e-3) * 1e-9,
-                "kernel_gbs_compulsory": k2["bytes_compulsory"] / (k2["ms_total"] * 1e-3) * 1e-9,
-                "kernel_gflops": k2["flops"] / (k2["ms_total"] * 1e-3) * 1e-9,
-                "frac_of_measured_hbm": (k2["bytes_compulsory"] / (k2["ms_total"] * 1e-3) * 1e-9) / peak,
-            }
-            del fin, fout
+            dslash[name] = matpc_numbers(ctx, prec, recon)
+        # the paper's "solver runs 10-20% slower than the matvec" (P:556-558): one BiCGstab
+        # iteration (2 Mhat + BLAS) of the timed solves against 2 bare Mhat applications
+        it_ms = ms / max(iters, 1)
+        dslash["solver_vs_matpc"] = {"iteration_ms": it_ms, "two_matpc_ms": 2e-3 * dslash["fp32-12"]["matpc_us_median"],
+                                     "solver_slower_by": it_ms / (2e-3 * dslash["fp32-12"]["matpc_us_median"]) - 1,
+                                     "note": "step time incl. reliable updates, Schur prepare/reconstruct and the "
+                                             "final fp64 residual, per iteration"}
+        if N > 1:
+            # weak-scaling reference on the same box: each rank's local lattice on ONE GPU through the
+            # unsplit (no-communication) path, and the split path with the overlap switched off
+            one = qudax.Context(local_dims, device=local)
+            one.gauge_load(qgen.gauge(local_dims, GAUGE_SEED, eps=EPS), KAPPA, CSW, prec=4, recon=12, t_boundary=-1)
+            n1 = matpc_numbers(one, 4, 12)
+            one.close()
+            dslash["weak_scaling_fp32-12"] = {
+                "matpc_gflops_N": dslash["fp32-12"]["matpc_gflops_total"],
+                "matpc_gflops_1gpu_unsplit": n1["matpc_gflops_per_gpu"],
+                "efficiency": dslash["fp32-12"]["matpc_gflops_total"] / (N * n1["matpc_gflops_per_gpu"]),
+                "note": "GFLOPS_N / (N x GFLOPS_1), 1-GPU baseline = the unsplit kernel on the per-GPU lattice"}
+            if args.halo == "comm":
+                nov = qudax.Context(dims, nranks=N, rank=rank, device=local, comm=qudax.COMM_NCCL,
+                                    nccl_id=obj2[0], overlap=False, proc_grid=grid)
+                Ub = qgen.gauge_box(dims, GAUGE_SEED, origin, local_dims, eps=EPS)
+                nov.gauge_load(Ub, KAPPA, CSW, prec=4, recon=12, t_boundary=-1)
+                del Ub
+                dslash["fp32-12 overlap off"] = matpc_numbers(nov, 4, 12)
+                nov.close()
     solve_time = None
     if not args.no_extra and N == 1:
         dslash.update(single_gpu_extras(ctx, b_dev, peak))
+        dslash["config2 L2-resident"] = config2_l2_resident(peak)
         solve_time = config3_solve_time()
 
     # ---- CPU baseline: the oracle on the host cores (rank 0, N = 1 only)
@@ -457,6 +569,9 @@ def main():
         if one:
             cpu["one_thread"] = {"value": one["value"], "cores": one["cores"], "sample": one["sample"],
                                  "seconds": one["seconds"]}
+        if not args.no_extra:
+            cpu["oracle_operators"] = oracle_operator_seconds()
+            cpu["oracle_operators_1thread"] = oracle_operator_seconds_1thread()
 
     ctx.close()
     if rank == 0:

@@ -23,8 +23,9 @@ Field conventions: gauge U[4, T, Z, Y, X, 3, 3] (mu = x, y, z, t); spinor psi[T,
 4, 3] in the DeGrand-Rossi basis; parity of a site = (x + y + z + t) mod 2 (reading Q14);
 a "parity field" is a full-lattice array that is zero on the other parity.
 
-Parity status: every function here is pinned by tests/test_oracle_*.py (see DESIGN.md
-§Oracle pins); none is "parity unpinned".
+Parity status: every function here is pinned by tests/test_oracle_pins.py (DESIGN.md §3 lists
+each function with its pin; apply_M_chunked by test_apply_M_chunked_pins); none is "parity
+unpinned".
 """
 import ctypes
 import os

@@ -313,6 +313,9 @@ static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res);
 // whether a reduction's local sums must go through the transport before they are used: several
 // ranks, or the NCCL loopback at one rank (which runs the N > 1 code path on one GPU)
 static bool global_sums(const qudax_ctx *c) { return c->g.nranks > 1 || c->comm == QUDAX_COMM_NCCL; }
+// whether that global sum happens after the kernel (transport) rather than inside its reduction
+// tail (the P2P mode's kernel-side allreduce, DevAllreduce)
+static bool sums_after_kernel(const qudax_ctx *c) { return global_sums(c) && !c->dar; }
 
 static cudaEvent_t pool_event(qudax_ctx *c) {
     if (!c->ev_pool.empty()) {
@@ -406,7 +409,7 @@ void harvest_graph_timing(qudax_ctx *c, const std::vector<qudax_ctx::TimingRec> 
 void check_device_error(qudax_ctx *c) {
     if (c->h_err && *reinterpret_cast<volatile int *>(c->h_err)) {
         *reinterpret_cast<volatile int *>(c->h_err) = 0;
-        throw Error(QUDAX_ERR_COMM, "kernel-initiated halo: a neighbour's face flag did not arrive (wait timed out); "
+        throw Error(QUDAX_ERR_COMM, "kernel-initiated halo or allreduce: a peer flag did not arrive (wait timed out); "
                                     "the operator result is invalid");
     }
 }
@@ -474,7 +477,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
     const long n_int = g.n_int, n_bnd = g.Vh - g.n_int;
     const bool split = c->comm == QUDAX_COMM_NCCL && !c->p2p.on && c->overlap && n_int > 0;
-    const bool multi = global_sums(c);  // sums go through the transport before the recurrence
+    const bool multi = sums_after_kernel(c);  // sums go through the transport before the recurrence
     if (red) {
         QX_CHECK(red->kind != RED_XDOT_NORM || kind >= QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
         QX_CHECK(red->kind != RED_RHAT_DOT || red->rhat, QUDAX_ERR_ARG, "rhat-dot needs rhat");
@@ -490,6 +493,8 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         args.tail.out = red->S ? red->S->red : c->red_out;
         args.tail.S = red->S;
         args.tail.coef_mode = (red->S && !multi) ? red->coef_mode : COEF_NONE;
+        args.tail.dar = c->dar;
+        args.tail.chan = 0;
     }
     auto launch = [&](int range, int nthreads) {
         args.range = range;
@@ -656,7 +661,11 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
         QX_CHECK(out[k] && in[k] && (kind < QUDAX_CLOVER_XPAY || (x && x[k])), QUDAX_ERR_ARG, "null field");
         QX_CHECK(out[k] != in[k], QUDAX_ERR_ARG, "dslash cannot run in place");
     }
-    if (c->comm != QUDAX_COMM_NONE || c->p2p.on || n == 1) {
+    const Geom &g = c->g;
+    // partitioned contexts: the multi-RHS halo (T-only split, comm transport) — one exchange per
+    // direction carrying every right-hand side's face — else one single-RHS operator per field
+    const bool mhalo = (c->comm != QUDAX_COMM_NONE) && !c->p2p.on && g.split == 8;
+    if ((c->comm != QUDAX_COMM_NONE && !mhalo) || c->p2p.on || n == 1) {
         for (int k = 0; k < n; ++k)
             dslash_op(c, out[k], in[k], x ? x[k] : nullptr, prec, p, dagger, kind, a, reds ? reds + k : nullptr, reverse);
         return;
@@ -669,8 +678,10 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
         args.out_m[k] = out[k];
         args.x_m[k] = x ? x[k] : nullptr;
     }
+    const bool multi = sums_after_kernel(c);
+    const long n_int = g.n_int, n_bnd = g.Vh - g.n_int;
+    const bool split = mhalo && c->comm == QUDAX_COMM_NCCL && c->overlap && n_int > 0;
     if (reds) {  // one deterministic reduction (and scalar recurrence) per right-hand side
-        const Geom &g = c->g;
         const int nb = dslash_blocks_any(prec, gc.recon, dagger, kind, (int)g.Vh);
         const size_t slots = 3 * ((size_t)nb + nb / kGroupHost + 2);
         const size_t ncount = 2 + (size_t)nb / kGroupHost + 2;
@@ -685,15 +696,77 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
             QX_CHECK(reds[k].kind != RED_XDOT_NORM || kind >= QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
             QX_CHECK(reds[k].kind != RED_RHAT_DOT || reds[k].rhat, QUDAX_ERR_ARG, "rhat-dot needs rhat");
             args.rhat_m[k] = reds[k].rhat;
-            args.tail_m[k] = RedTail{c->dpart_m + slots * k, c->dcount_m + ncount * k, nb, 0, reds[k].S->red, reds[k].S,
-                                     reds[k].coef_mode};
+            const int tot = split ? dslash_blocks_any(prec, gc.recon, dagger, kind, (int)n_int) +
+                                        dslash_blocks_any(prec, gc.recon, dagger, kind, (int)n_bnd)
+                                  : nb;
+            args.tail_m[k] = RedTail{c->dpart_m + slots * k, c->dcount_m + ncount * k, tot, 0, reds[k].S->red, reds[k].S,
+                                     multi ? COEF_NONE : reds[k].coef_mode, c->dar, 1 + k};
         }
     }
-    args.ghosted = 0;
-    args.range = RANGE_ALL;
-    args.nthreads = (int)c->g.Vh;
-    launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
-    c->launches += 1;
+    int blk_off = 0;
+    auto launch = [&](int range, int nthreads) {
+        args.range = range;
+        args.nthreads = nthreads;
+        for (int k = 0; k < n; ++k) args.tail_m[k].block_offset = blk_off;
+        launch_dslash_ctx(c, prec, gc.recon, dagger, kind, args);
+        blk_off += dslash_blocks_any(prec, gc.recon, dagger, kind, nthreads);
+        c->launches += 1;
+    };
+    if (!mhalo) {
+        args.ghosted = 0;
+        launch(RANGE_ALL, (int)g.Vh);
+        return;
+    }
+    // ---- multi-RHS T halo (P:692-720 with every right-hand side in one message per direction)
+    auto &h = halo_for(c, prec);
+    const bool host = c->comm == QUDAX_COMM_HOST;
+    if (!h.m_sb) {
+        h.m_stride = (h.bytes + 255) & ~(size_t)255;
+        const size_t mb = h.m_stride * kMaxRhs;
+        h.m_sb = dalloc(c, mb);
+        h.m_sf = dalloc(c, mb);
+        h.m_gb = dalloc(c, mb);
+        h.m_gf = dalloc(c, mb);
+        if (host) {
+            h.mh_sb = halloc(c, mb);
+            h.mh_sf = halloc(c, mb);
+            h.mh_gb = halloc(c, mb);
+            h.mh_gf = halloc(c, mb);
+        }
+    }
+    args.ghosted = 1;
+    args.ghost_back = h.m_gb;
+    args.ghost_fwd = h.m_gf;
+    args.ghost_rhs_bytes = (long)h.m_stride;
+    Xfer xf{3, h.m_sf, h.m_sb, h.m_gb, h.m_gf, h.m_stride * n, h.mh_sf, h.mh_sb, h.mh_gb, h.mh_gf};
+    auto pack_all = [&](cudaStream_t st) {
+        for (int k = 0; k < n; ++k) {
+            launch_pack_faces(prec, dagger, g, in[k], static_cast<char *>(h.m_sb) + k * h.m_stride,
+                              static_cast<char *>(h.m_sf) + k * h.m_stride, c->halt, st);
+            c->launches += 1;
+        }
+    };
+    if (c->comm == QUDAX_COMM_NCCL) {
+        QX_CUDA(cudaEventRecord(c->ev_in, c->stream));
+        QX_CUDA(cudaStreamWaitEvent(c->comm_stream, c->ev_in, 0));
+        pack_all(c->comm_stream);
+        exchange_all(c, &xf, 1, c->comm_stream);
+        QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
+        if (split) {
+            launch(RANGE_INTERIOR, (int)n_int);
+            QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
+            launch(RANGE_BOUNDARY, (int)n_bnd);
+        } else {
+            QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
+            launch(RANGE_ALL, (int)g.Vh);
+        }
+    } else {  // HOST transport: exchange first, one launch
+        pack_all(c->stream);
+        exchange_all(c, &xf, 1, c->stream);
+        launch(RANGE_ALL, (int)g.Vh);
+    }
+    if (reds && multi)
+        for (int k = 0; k < n; ++k) device_sum_coef(c, reds[k].S->red, 3, reds[k].S, reds[k].coef_mode);
 }
 
 void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger,
@@ -718,6 +791,13 @@ void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int pari
 }
 
 static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res) {
+    if (c->dar) {  // the kernel's reduction tail already summed over ranks (DevAllreduce)
+        QX_CUDA(cudaMemcpyAsync(c->h_red, dev_vals, sizeof(double) * n, cudaMemcpyDeviceToHost, c->stream));
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        check_device_error(c);
+        for (int k = 0; k < n; ++k) res[k] = c->h_red[k];
+        return;
+    }
     if (c->comm == QUDAX_COMM_NCCL) {  // (one rank: the loopback test of the N > 1 path)
         QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl, c->stream));
     }
@@ -735,7 +815,7 @@ int blas_op(qudax_ctx *c, int op, int prec, void *const *f, const double *coef, 
         co[0].v = make_double2(coef[0], op == OP_XPAY ? 0.0 : coef[1]);
         if (op == OP_P_UPDATE || op == OP_FINAL) co[1].v = make_double2(coef[2], coef[3]);
     }
-    RedTail tail{c->partials, c->d_counter, 0, 0, c->red_out, nullptr, COEF_NONE};
+    RedTail tail{c->partials, c->d_counter, 0, 0, c->red_out, nullptr, COEF_NONE, c->dar, 0};
     int n = blas_run(op, prec, c->g, f, co, tail, c->halt, c->stream);
     c->launches += 1;
     if (n) global_sum(c, c->red_out, n, res);
@@ -762,8 +842,8 @@ void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, in
 // BLAS op whose coefficients may live on the device; its reduction (if any) goes to S->red,
 // is summed over ranks and fed to the scalar recurrence `mode` — all stream-ordered.
 void blas_op_dev(qudax_ctx *c, int op, int prec, void *const *f, const CoefArg *co, SolverScalars *S, int mode) {
-    const bool multi = global_sums(c);
-    RedTail tail{c->partials, c->d_counter, 0, 0, S->red, S, multi ? COEF_NONE : mode};
+    const bool multi = sums_after_kernel(c);
+    RedTail tail{c->partials, c->d_counter, 0, 0, S->red, S, multi ? COEF_NONE : mode, c->dar, 0};
     int n = blas_run(op, prec, c->g, f, co, tail, c->halt, c->stream);
     c->launches += 1;
     if (n && multi) device_sum_coef(c, S->red, n, S, mode);
@@ -1065,8 +1145,43 @@ qudax_status qudax_nccl_unique_id(void *out128) {
     return QUDAX_OK;
 }
 
+// Allgather of one small record per rank over the comm transport: NCCL (device buffers), or the
+// host hooks — the allreduce hook sums doubles, so each rank places its bytes, as exact 16-bit
+// integers, in its own slice of a zero array (sums of one non-zero term are exact).
+static void allgather_small(qudax_ctx *c, const void *mine, size_t n, void *all) {
+    const Geom &g = c->g;
+    if (c->comm == QUDAX_COMM_NCCL) {
+        char *d = static_cast<char *>(dalloc(c, n * (g.nranks + 1)));
+        QX_CUDA(cudaMemcpyAsync(d, mine, n, cudaMemcpyHostToDevice, c->stream));
+        QX_NCCL(ncclAllGather(d, d + n, n, ncclChar, c->nccl, c->stream));
+        QX_CUDA(cudaMemcpyAsync(all, d + n, n * g.nranks, cudaMemcpyDeviceToHost, c->stream));
+        QX_CUDA(cudaStreamSynchronize(c->stream));
+        dfree(c, d);
+    } else if (c->comm == QUDAX_COMM_HOST) {
+        const size_t w = (n + 1) / 2;  // 16-bit words per record
+        std::vector<double> v(w * g.nranks, 0.0);
+        const unsigned char *m = static_cast<const unsigned char *>(mine);
+        for (size_t k = 0; k < w; ++k)
+            v[w * g.rank + k] = (double)(m[2 * k] | ((2 * k + 1 < n ? m[2 * k + 1] : 0) << 8));
+        if (c->host_allreduce(v.data(), (int)v.size(), c->comm_user))
+            throw Error(QUDAX_ERR_COMM, "host_allreduce hook failed (allgather)");
+        unsigned char *o = static_cast<unsigned char *>(all);
+        for (int r = 0; r < g.nranks; ++r)
+            for (size_t k = 0; k < n; ++k) {
+                const unsigned u = (unsigned)v[w * r + k / 2];
+                o[n * r + k] = (unsigned char)((k & 1) ? (u >> 8) : (u & 255));
+            }
+    } else {
+        throw Error(QUDAX_ERR_ARG, "P2P mode with nranks > 1 needs a comm transport for the handle exchange");
+    }
+}
+
 // QUDAX_HALO_P2P setup: one IPC-exportable region per rank with the same layout everywhere
-// (ctx.h P2P), its handle swapped with both T-neighbours over the comm transport, theirs mapped.
+// (ctx.h P2P): the halo ghosts and flags, and the slot area of the kernel-side allreduce
+// (internal.h DevAllreduce).  Every rank's {IPC handle, PCI bus id} is allgathered; the
+// T-neighbours' regions (and, for nranks <= kMaxPeers, every rank's, for the allreduce) are
+// mapped.  A rank on another GPU must be reachable by peer access (NVLink / NVSwitch on a B200
+// node), else UNSUPPORTED: the comm path (NCCL) is for GPUs without peer access.
 static void setup_p2p(qudax_ctx *c) {
     auto &q = c->p2p;
     const Geom &g = c->g;
@@ -1086,66 +1201,66 @@ static void setup_p2p(qudax_ctx *c) {
     q.off_count = cur + 128;
     q.off_cseq = cur + 192;
     q.off_ccount = cur + 256;
-    q.bytes = cur + 512;
+    q.off_ar = cur + 512;
+    q.bytes = q.off_ar + sizeof(double) * 4 * kArChannels * 2 * kMaxPeers;
     void *base = nullptr;
     QX_CUDA(cudaMalloc(&base, q.bytes));  // not the caller's allocator: IPC exports whole allocations
     q.base = static_cast<char *>(base);
     QX_CUDA(cudaMemset(q.base, 0, q.bytes));
     QX_CUDA(cudaDeviceSynchronize());
-    if (g.nranks == 1) {  // loopback: the neighbour is this rank
-        q.peer_back = q.peer_fwd = q.base;
-        return;
-    }
-    static_assert(sizeof(cudaIpcMemHandle_t) == 64, "IPC handle size");
-    // each rank sends {IPC handle, PCI bus id of its GPU}: a neighbour on another GPU must be
-    // reachable by peer access (NVLink / NVSwitch on a B200 node), else UNSUPPORTED — the comm
-    // halo (NCCL) is the path for GPUs without peer access
-    struct Rec {
-        cudaIpcMemHandle_t h;
-        char bus[64];
-    };
-    Rec mine{}, rb{}, rf{};
-    QX_CUDA(cudaIpcGetMemHandle(&mine.h, q.base));
-    QX_CUDA(cudaDeviceGetPCIBusId(mine.bus, sizeof(mine.bus), c->device));
-    if (c->comm == QUDAX_COMM_HOST) {
-        Rec s0 = mine, s1 = mine;
-        if (c->host_exchange(g.nbf[3], g.nbb[3], &s0, &s1, &rb, &rf, sizeof(Rec), c->comm_user))
-            throw Error(QUDAX_ERR_COMM, "host_exchange hook failed (IPC handles)");
-    } else if (c->comm == QUDAX_COMM_NCCL) {
-        char *d = static_cast<char *>(dalloc(c, 3 * sizeof(Rec)));
-        QX_CUDA(cudaMemcpyAsync(d, &mine, sizeof(Rec), cudaMemcpyHostToDevice, c->stream));
-        exchange(c, d, d, d + sizeof(Rec), d + 2 * sizeof(Rec), sizeof(Rec), c->stream, nullptr, nullptr, nullptr,
-                 nullptr);
-        QX_CUDA(cudaMemcpyAsync(&rb, d + sizeof(Rec), sizeof(Rec), cudaMemcpyDeviceToHost, c->stream));
-        QX_CUDA(cudaMemcpyAsync(&rf, d + 2 * sizeof(Rec), sizeof(Rec), cudaMemcpyDeviceToHost, c->stream));
-        QX_CUDA(cudaStreamSynchronize(c->stream));
-        dfree(c, d);
-    } else {
-        throw Error(QUDAX_ERR_ARG, "P2P halo with nranks > 1 needs a comm transport for the handle exchange");
-    }
-    for (const Rec *r : {&rb, &rf}) {
-        if (std::strncmp(r->bus, mine.bus, sizeof(mine.bus)) == 0) continue;  // same GPU (test mode)
-        int peer = -1, can = 0;
-        if (cudaDeviceGetByPCIBusId(&peer, r->bus) != cudaSuccess) {
-            cudaGetLastError();  // the peer GPU is not visible to this process: no peer access
-            throw Error(QUDAX_ERR_UNSUPPORTED, std::string("P2P halo: neighbour GPU ") + r->bus + " not visible here");
+    for (int r = 0; r < kMaxPeers; ++r) q.peer[r] = nullptr;
+    if (g.nranks > 1) {
+        static_assert(sizeof(cudaIpcMemHandle_t) == 64, "IPC handle size");
+        struct Rec {
+            cudaIpcMemHandle_t h;
+            char bus[64];
+        };
+        Rec mine{};
+        QX_CUDA(cudaIpcGetMemHandle(&mine.h, q.base));
+        QX_CUDA(cudaDeviceGetPCIBusId(mine.bus, sizeof(mine.bus), c->device));
+        std::vector<Rec> all(g.nranks);
+        allgather_small(c, &mine, sizeof(Rec), all.data());
+        const bool map_all = g.nranks <= kMaxPeers;
+        q.opened.assign(g.nranks, nullptr);
+        for (int r = 0; r < g.nranks; ++r) {
+            if (r == g.rank || !(map_all || r == g.nbf[3] || r == g.nbb[3])) continue;
+            const Rec &rec = all[r];
+            if (std::strncmp(rec.bus, mine.bus, sizeof(mine.bus)) != 0) {  // another GPU (else test mode)
+                int peer = -1, can = 0;
+                if (cudaDeviceGetByPCIBusId(&peer, rec.bus) != cudaSuccess) {
+                    cudaGetLastError();  // the peer GPU is not visible to this process: no peer access
+                    throw Error(QUDAX_ERR_UNSUPPORTED, std::string("P2P: rank ") + std::to_string(r) + "'s GPU " +
+                                                           rec.bus + " not visible here");
+                }
+                QX_CUDA(cudaDeviceCanAccessPeer(&can, c->device, peer));
+                if (!can)
+                    throw Error(QUDAX_ERR_UNSUPPORTED, std::string("P2P: no peer access to rank ") + std::to_string(r) +
+                                                           "'s GPU " + rec.bus);
+            }
+            void *pr = nullptr;
+            QX_CUDA(cudaIpcOpenMemHandle(&pr, rec.h, cudaIpcMemLazyEnablePeerAccess));
+            q.opened[r] = static_cast<char *>(pr);
         }
-        QX_CUDA(cudaDeviceCanAccessPeer(&can, c->device, peer));
-        if (!can)
-            throw Error(QUDAX_ERR_UNSUPPORTED, std::string("P2P halo: no peer access to neighbour GPU ") + r->bus);
+        auto region = [&](int r) { return r == g.rank ? q.base : q.opened[r]; };
+        q.peer_back = region(g.nbb[3]);
+        q.peer_fwd = region(g.nbf[3]);
+        if (map_all)
+            for (int r = 0; r < g.nranks; ++r) q.peer[r] = region(r);
+    } else {  // loopback: the neighbour is this rank
+        q.peer_back = q.peer_fwd = q.base;
+        q.peer[0] = q.base;
     }
-    const cudaIpcMemHandle_t hb = rb.h, hf = rf.h;
-    void *pb = nullptr;
-    QX_CUDA(cudaIpcOpenMemHandle(&pb, hb, cudaIpcMemLazyEnablePeerAccess));
-    q.peer_back = static_cast<char *>(pb);
-    q.opened_back = true;
-    if (rank_fwd(g) == rank_back(g)) {  // two ranks: one neighbour on both sides
-        q.peer_fwd = q.peer_back;
-    } else {
-        void *pf = nullptr;
-        QX_CUDA(cudaIpcOpenMemHandle(&pf, hf, cudaIpcMemLazyEnablePeerAccess));
-        q.peer_fwd = static_cast<char *>(pf);
-        q.opened_fwd = true;
+    // kernel-side allreduce descriptor (device memory), when every rank is mapped
+    if (g.nranks <= kMaxPeers) {
+        DevAllreduce d{};
+        for (int r = 0; r < g.nranks; ++r) d.slots[r] = reinterpret_cast<double *>(q.peer[r] + q.off_ar);
+        d.seq = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * kArChannels));
+        QX_CUDA(cudaMemset(d.seq, 0, sizeof(unsigned) * kArChannels));
+        d.nranks = g.nranks;
+        d.rank = g.rank;
+        d.err = c->d_err;
+        c->dar = static_cast<DevAllreduce *>(dalloc(c, sizeof(DevAllreduce)));
+        QX_CUDA(cudaMemcpy(c->dar, &d, sizeof(d), cudaMemcpyHostToDevice));
     }
 }
 
@@ -1286,8 +1401,8 @@ qudax_status qudax_finalize(qudax_ctx *c) {
                          std::get<1>(kv.first), std::get<2>(kv.first), kv.second.first, 1e3 * kv.second.second / kv.second.first);
     if (c->stream) cudaStreamSynchronize(c->stream);
     if (c->comm_stream) cudaStreamSynchronize(c->comm_stream);
-    if (c->p2p.opened_fwd) cudaIpcCloseMemHandle(c->p2p.peer_fwd);
-    if (c->p2p.opened_back) cudaIpcCloseMemHandle(c->p2p.peer_back);
+    for (char *m : c->p2p.opened)
+        if (m) cudaIpcCloseMemHandle(m);
     if (c->p2p.base) cudaFree(c->p2p.base);
     if (c->nccl) ncclCommDestroy(c->nccl);
     for (void *p : c->allocs) {

@@ -95,6 +95,11 @@ struct qudax_ctx {
         size_t sbytes[3] = {};
         void *ssb[3] = {}, *ssf[3] = {}, *sgb[3] = {}, *sgf[3] = {};
         void *h_ssb[3] = {}, *h_ssf[3] = {}, *h_sgb[3] = {}, *h_sgf[3] = {};
+        // multi-RHS T halo: kMaxRhs faces per buffer, RHS k at k * m_stride (one message per
+        // direction carries every right-hand side)
+        size_t m_stride = 0;
+        void *m_sb = nullptr, *m_sf = nullptr, *m_gb = nullptr, *m_gf = nullptr;
+        void *mh_sb = nullptr, *mh_sf = nullptr, *mh_gb = nullptr, *mh_gf = nullptr;
     } halo[3];
     int *blist = nullptr;  // boundary sites (complement of the interior box) when X/Y/Z is split
 
@@ -107,10 +112,13 @@ struct qudax_ctx {
         bool on = false;
         char *base = nullptr;                       // own region (cudaMalloc, IPC-exported)
         char *peer_back = nullptr, *peer_fwd = nullptr;  // neighbours' regions (IPC-mapped or own)
-        bool opened_back = false, opened_fwd = false;
+        char *peer[qx::kMaxPeers] = {};                  // every rank's region (nranks <= kMaxPeers)
+        std::vector<char *> opened;                      // IPC mappings to close at finalize
         size_t off_gb[3] = {}, off_gf[3] = {}, pdist[3] = {};
-        size_t off_flags = 0, off_seq = 0, off_count = 0, off_cseq = 0, off_ccount = 0, bytes = 0;
+        size_t off_flags = 0, off_seq = 0, off_count = 0, off_cseq = 0, off_ccount = 0, off_ar = 0, bytes = 0;
     } p2p;
+    // kernel-side allreduce descriptor (device memory) of the P2P mode, nullptr otherwise
+    qx::DevAllreduce *dar = nullptr;
 
     // workspace
     void *tmp_odd[3] = {}, *tmp_even[3] = {}, *tmp_sym[3] = {};

@@ -459,6 +459,20 @@ __host__ __device__ constexpr bool dslash_pair() {
     return P == 8 || (P == 2 && RECON != 12);
 #endif
 }
+// Whether the unpartitioned kernel runs its 8 hops as a software pipeline: the raw operands of
+// hop k+1 (neighbour spinor + link, still packed) are loaded before hop k is decoded and
+// computed, so one hop's loads are always in flight (dslash_pair only overlaps the two hops of
+// one direction, then waits).  The half kernel was memory-latency bound at its register-capped
+// occupancy (ncu r01k: stall samples on the first PRMT after every hop's loads).
+// QX_PIPE_MASK overrides: bit 0 half, 1 fp32, 2 fp64.
+template <int P, int RECON>
+__host__ __device__ constexpr bool dslash_pipe() {
+#ifdef QX_PIPE_MASK
+    return (QX_PIPE_MASK >> (P == 2 ? 0 : (P == 4 ? 1 : 2))) & 1;
+#else
+    return P == 2;
+#endif
+}
 #ifndef QX_DSLASH_THREADS
 #define QX_DSLASH_THREADS 128
 #endif
@@ -674,12 +688,107 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             spatial_hop<MU, SB, true, DF>(ps, u, acc, sc);
         }
     };
-    spatial(std::integral_constant<int, 0>{}, x, X, (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1,
-            (x == 0 ? lex + (X - 1) : lex - 1) >> 1);
-    spatial(std::integral_constant<int, 1>{}, y, Y, (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1,
-            (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1);
-    spatial(std::integral_constant<int, 2>{}, z, Z, (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1,
-            (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1);
+    // neighbour checkerboard indices of the six spatial hops (periodic wrap inside the box)
+    const int nxf = (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1, nxb = (x == 0 ? lex + (X - 1) : lex - 1) >> 1;
+    const int nyf = (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1, nyb = (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1;
+    const int nzf = (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1, nzb = (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1;
+    constexpr bool PIPE = !SS && dslash_pipe<P, RECON>();
+    if constexpr (PIPE) {
+        // ---- software-pipelined hops (dslash_pipe): load hop k+1, then compute hop k
+        const int T_loc = a.T_loc;
+        constexpr bool FWD_UPPER = (SF > 0), BWD_UPPER = (SB > 0);
+        const bool fwd_ghost = (t == T_loc - 1) && a.ghosted;
+        const bool bwd_ghost = (t == 0) && a.ghosted;
+        const R cft = (t == T_loc - 1) ? (R)(2.0 * a.bc_fwd) : (R)2;
+        const R cbt = (t == 0) ? (R)(2.0 * a.bc_back) : (R)2;
+        const int nfw = (t == T_loc - 1 ? lex - (T_loc - 1) * XYZ : lex + XYZ) >> 1;
+        const int nbw = (t == 0 ? lex + (T_loc - 1) * XYZ : lex - XYZ) >> 1;
+        struct SpHop {
+            RawVec<P, 24> s;
+            RawLink<P, RECON> l;
+        };
+        struct THop {
+            RawVec<P, 12> s;
+            RawLink<P, RECON> l;
+        };
+        auto load_sp = [&](SpHop &h, int mu, bool fwd, int n) {
+            h.s.template load_spinor<INMODE>(fin, a.stride, n);
+            if (fwd) h.l.load(a.gauge[mu][p], a.stride, i);
+            else h.l.load(a.gauge[mu][op], a.stride, n);
+        };
+        auto comp_sp = [&](const SpHop &h, auto mu_c, auto sg_c) {
+            constexpr int MU = decltype(mu_c)::value, SG = decltype(sg_c)::value;
+            constexpr bool ADJ = (SG == SB);  // the backward hop applies U(x - mu)^dag
+            R v[24];
+            Cx<R> ps[4][3], u[3][3];
+            if constexpr (DF && QX_BPROJ) {
+                Cx<R> h0[3], h1[3];
+                h.s.decode_b(v);
+                unpack_spinor(v, ps);
+                spatial_project_b<MU, SG>(ps, h0, h1);
+                const R sc = h.s.scale() * dec_link<DF>(h.l, u);
+                spatial_mult_expand<MU, SG, ADJ, DF>(h0, h1, u, acc, sc);
+            } else {
+                R sc = dec_vec<DF>(h.s, v);
+                unpack_spinor(v, ps);
+                sc *= dec_link<DF>(h.l, u);
+                spatial_hop<MU, SG, ADJ, DF>(ps, u, acc, sc);
+            }
+        };
+        auto load_tf = [&](THop &h) {
+            if (fwd_ghost) h.s.load_face(static_cast<const char *>(a.ghost_fwd) + goff, a.fstride, i - t * a.F);
+            else h.s.template load_half<INMODE>(fin, a.stride, nfw, FWD_UPPER ? 0 : 1);
+            h.l.load(a.gauge[3][p], a.stride, i);
+        };
+        auto load_tb = [&](THop &h) {
+            if (bwd_ghost) {
+                h.s.load_face(static_cast<const char *>(a.ghost_back) + goff, a.fstride, i);
+                h.l.load(a.gauge_ghost, a.fstride, i);
+            } else {
+                h.s.template load_half<INMODE>(fin, a.stride, nbw, BWD_UPPER ? 0 : 1);
+                h.l.load(a.gauge[3][op], a.stride, nbw);
+            }
+        };
+        auto comp_t = [&](const THop &h, auto up_c, auto adj_c, R coef) {
+            R hv[12];
+            Cx<R> u[3][3];
+            R sc = dec_vec<DF>(h.s, hv);
+            sc *= dec_link<DF>(h.l, u);
+            temporal_hop<decltype(up_c)::value, decltype(adj_c)::value>(hv, u, DF ? coef * sc : coef, acc);
+        };
+        using I0 = std::integral_constant<int, 0>;
+        using I1 = std::integral_constant<int, 1>;
+        using I2 = std::integral_constant<int, 2>;
+        using CF = std::integral_constant<int, SF>;
+        using CB = std::integral_constant<int, SB>;
+        SpHop A, B;
+        load_sp(A, 0, true, nxf);
+        load_sp(B, 0, false, nxb);
+        comp_sp(A, I0{}, CF{});
+        load_sp(A, 1, true, nyf);
+        comp_sp(B, I0{}, CB{});
+        load_sp(B, 1, false, nyb);
+        comp_sp(A, I1{}, CF{});
+        load_sp(A, 2, true, nzf);
+        comp_sp(B, I1{}, CB{});
+        load_sp(B, 2, false, nzb);
+        comp_sp(A, I2{}, CF{});
+        THop C, D;
+        load_tf(C);
+        comp_sp(B, I2{}, CB{});
+        load_tb(D);
+#if QX_RED_PF
+        if (a.red_kind != RED_NONE) {
+            const void *w = a.red_kind == RED_XDOT_NORM ? fx : (a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat);
+            pf_spinor_l1<P>(w, a.stride, i);
+        }
+#endif
+        comp_t(C, std::bool_constant<FWD_UPPER>{}, std::false_type{}, cft);
+        comp_t(D, std::bool_constant<BWD_UPPER>{}, std::true_type{}, cbt);
+    } else {
+    spatial(std::integral_constant<int, 0>{}, x, X, nxf, nxb);
+    spatial(std::integral_constant<int, 1>{}, y, Y, nyf, nyb);
+    spatial(std::integral_constant<int, 2>{}, z, Z, nzf, nzb);
 
     // ---- t direction: diagonal projectors, 12 reals per neighbour (eq. (6))
     {
@@ -738,6 +847,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             temporal_hop<BWD_UPPER, true>(h, u, DF ? cb * sc : cb, acc);
         }
     }
+    }  // !PIPE
 
     // ---- epilogue: fused clover
     Cx<R> res[4][3];
@@ -857,7 +967,7 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     const void *fin = a.nrhs > 1 ? a.in_m[rhs] : a.in;
     void *fout = a.nrhs > 1 ? a.out_m[rhs] : a.out;
     const void *fx = a.nrhs > 1 ? a.x_m[rhs] : a.x;
-    long goff = 0;
+    long goff = (long)rhs * a.ghost_rhs_bytes;  // multi-RHS halo: this RHS's ghost faces
     // RANGE_TAIL: only CTAs holding boundary sites (the grid's last ones) wait for the halo
     if (a.p2p_flags && (a.range != RANGE_TAIL || (blk + 1) * (int)blockDim.x > (a.T_loc - 2) * a.F)) goff = p2p_wait(a);
     if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND, 0, SS>(a, fin, fout, fx, tid, red, goff);

@@ -7,8 +7,9 @@
 // site for NR right-hand sides: each link is loaded and reconstructed once and applied to the
 // NR neighbour spinors, each clover block once for the NR vectors.  Same arithmetic per RHS as
 // dslash_site (same helpers, same operation order), so the result is bitwise the single-RHS
-// one.  Unpartitioned lattices only (RANGE_ALL, no ghosts); an odd last group repeats its
-// last RHS and skips its stores.
+// one.  Unpartitioned lattices, or T-partitioned ones with the multi-RHS halo (interior /
+// boundary ranges, one ghost face per RHS); an odd last group repeats its last RHS and skips its
+// stores.
 #pragma once
 #include "dslash.cuh"
 
@@ -64,12 +65,15 @@ __device__ __forceinline__ void apply_clover_mr(const void *cl, long stride, lon
 }
 
 template <int P, int RECON, bool DAG, int KIND, int NR>
-__device__ __forceinline__ void dslash_site_mr(const DslashArgs &a, int tid, const void *const *fin, void *const *fout,
-                                               const void *const *fx, const void *const *frh, bool last_valid,
-                                               double (*red)[3]) {
+__device__ __forceinline__ void dslash_site_mr(const DslashArgs &a, int tid, int r0, const void *const *fin,
+                                               void *const *fout, const void *const *fx, const void *const *frh,
+                                               bool last_valid, double (*red)[3]) {
     using R = typename Prec<P>::R;
     if (a.reverse) tid = a.nthreads - 1 - tid;
-    const int i = tid;
+    // T-partitioned contexts (multi-RHS halo): interior sites t in [1, T_loc-2], or the 2F
+    // boundary sites (t = 0 and t = T_loc-1), as in dslash_site
+    const int i = a.range == RANGE_ALL ? tid
+                  : (a.range == RANGE_INTERIOR ? a.F + tid : (tid < a.F ? tid : (a.T_loc - 1) * a.F + (tid - a.F)));
     const int X = a.X, Y = a.Y, Z = a.Z, Xh = a.Xh;
     int xh, y, z, t;
     {
@@ -171,7 +175,8 @@ __device__ __forceinline__ void dslash_site_mr(const DslashArgs &a, int tid, con
         hop(I2{}, PB{}, AD{}, a.gauge[2][op], nb, nb);
     }
     // t direction: diagonal projectors, 12 reals per neighbour (eq. (6)); periodic wrap with the
-    // boundary sign on the local (= global, unpartitioned) edge
+    // boundary sign on the local edge, or (T-partitioned, a.ghosted) the neighbours' faces: one
+    // halo carries every right-hand side, RHS k's face at k * a.ghost_rhs_bytes
     {
         constexpr bool FWD_UPPER = (SF > 0);
         constexpr bool BWD_UPPER = (SB > 0);
@@ -180,27 +185,40 @@ __device__ __forceinline__ void dslash_site_mr(const DslashArgs &a, int tid, con
         const R cb = (t == 0) ? (R)(2.0 * a.bc_back) : (R)2;
         const int nfw = (t == T_loc - 1 ? lex - (T_loc - 1) * XYZ : lex + XYZ) >> 1;
         const int nbw = (t == 0 ? lex + (T_loc - 1) * XYZ : lex - XYZ) >> 1;
-        auto thop = [&](auto up_c, auto adj_c, const void *lbase, int li, int n, R coef) {
+        const bool fwd_ghost = (t == T_loc - 1) && a.ghosted;
+        const bool bwd_ghost = (t == 0) && a.ghosted;
+        auto thop = [&](auto up_c, auto adj_c, bool ghost, const void *gbase, long gf, const void *lbase, long lstr,
+                        int li, int n, R coef) {
             constexpr bool UP = decltype(up_c)::value;
             constexpr bool ADJ = decltype(adj_c)::value;
             RawLink<P, RECON> l;
-            l.load(lbase, a.stride, li);
+            l.load(lbase, lstr, li);
+            auto ld = [&](RawVec<P, 12> &hv, int r) {
+                if (ghost) hv.load_face(static_cast<const char *>(gbase) + (long)(r0 + r) * a.ghost_rhs_bytes, a.fstride, gf);
+                else hv.template load_half<0>(fin[r], a.stride, n, UP ? 0 : 1);
+            };
             RawVec<P, 12> hv;
-            hv.template load_half<0>(fin[0], a.stride, n, UP ? 0 : 1);
+            ld(hv, 0);
             Cx<R> u[3][3];
             const R usc = dec_link<DF>(l, u);
 #pragma unroll
             for (int r = 0; r < NR; ++r) {
                 RawVec<P, 12> cur = hv;
-                if (r + 1 < NR) hv.template load_half<0>(fin[r + 1], a.stride, n, UP ? 0 : 1);
+                if (r + 1 < NR) ld(hv, r + 1);
                 R h[12];
                 R sc = dec_vec<DF>(cur, h);
                 sc *= usc;
                 temporal_hop<UP, ADJ>(h, u, DF ? coef * sc : coef, acc[r]);
             }
         };
-        thop(std::integral_constant<bool, FWD_UPPER>{}, NA{}, a.gauge[3][p], i, nfw, cf);
-        thop(std::integral_constant<bool, BWD_UPPER>{}, AD{}, a.gauge[3][op], nbw, nbw, cb);
+        thop(std::integral_constant<bool, FWD_UPPER>{}, NA{}, fwd_ghost, a.ghost_fwd, (long)(i - t * a.F),
+             a.gauge[3][p], a.stride, i, nfw, cf);
+        if (bwd_ghost)
+            thop(std::integral_constant<bool, BWD_UPPER>{}, AD{}, true, a.ghost_back, (long)i, a.gauge_ghost, a.fstride,
+                 i, nbw, cb);
+        else
+            thop(std::integral_constant<bool, BWD_UPPER>{}, AD{}, false, a.ghost_back, (long)i, a.gauge[3][op], a.stride,
+                 nbw, nbw, cb);
     }
 
     // epilogue: fused clover, store, optional per-RHS reductions
@@ -310,7 +328,7 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, DslashMrMinBlocks<P, NR>::v
     }
     const int tid = blk * blockDim.x + threadIdx.x;
     double red[NR][3] = {};
-    if (tid < a.nthreads) dslash_site_mr<P, RECON, DAG, KIND, NR>(a, tid, fin, fout, fx, frh, last_valid, red);
+    if (tid < a.nthreads) dslash_site_mr<P, RECON, DAG, KIND, NR>(a, tid, r0, fin, fout, fx, frh, last_valid, red);
     if (a.red_kind != RED_NONE) {
 #pragma unroll
         for (int r = 0; r < NR; ++r) {
@@ -325,7 +343,7 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, DslashMrMinBlocks<P, NR>::v
 template <int P>
 bool launch_dslash_mr_prec(int recon, int dagger, int kind, const DslashArgs &a, cudaStream_t s) {
     constexpr int NR = QX_MR_NR;
-    if (a.nrhs < 2 || a.smask || a.range != RANGE_ALL || a.p2p_flags) return false;
+    if (a.nrhs < 2 || a.smask || a.range == RANGE_TAIL || a.p2p_flags) return false;
     const int grid = ((a.nthreads + QX_DSLASH_THREADS - 1) / QX_DSLASH_THREADS) * ((a.nrhs + NR - 1) / NR);
 #define QX_MR(RC, DG, KD)                                                                             \
     if (recon == RC && dagger == DG && kind == KD) {                                                  \

@@ -103,6 +103,24 @@ struct SolverScalars {
     double hist[kHistRing];      // |r_k| (iterated) at ring slot (k - 1) % kHistRing
 };
 enum CoefMode { COEF_NONE = 0, COEF_ALPHA = 1, COEF_OMEGA = 2, COEF_RHO = 3 };
+// Kernel-side global sum over peer memory (QUDAX_HALO_P2P mode: the
+// solver's per-iteration sums fused with their allreduce): every rank owns one
+// IPC-exported slot area [kArChannels][2][kMaxPeers] of {3 sums, sequence}.  The CTA that
+// finishes a reduction stores its rank's totals into slot [chan][seq & 1][rank] of EVERY rank
+// (peer stores over NVLink, then a system-scope release of the sequence word), acquires the
+// nranks slots of its own area for this sequence, and adds them in rank order — so every rank
+// gets bitwise the same sums with no host involvement and no NCCL launch.  Channel = the
+// reduction stream (0: single-RHS, 1 + k: right-hand side k of a multi-RHS launch, whose tails
+// finish in any order); two sequence parities suffice because no rank can start sequence s + 2
+// of a channel before every rank has finished reading s (it needs their s + 1 totals first).
+constexpr int kMaxPeers = 8;
+constexpr int kArChannels = 1 + 8;  // 1 + kMaxRhs
+struct DevAllreduce {
+    double *slots[kMaxPeers];  // each rank's slot area (this rank's own at [rank]), peer-mapped
+    unsigned *seq;             // [kArChannels] this rank's per-channel sequence counters
+    int nranks, rank;
+    int *err;                  // device error word (wait timeout)
+};
 // a grid reduction with a last-CTA tail (reduce.cuh)
 struct RedTail {
     double *partials;      // [total_blocks][nred] per-CTA sums
@@ -112,6 +130,8 @@ struct RedTail {
     double *out;           // totals (S->red when coef_mode != COEF_NONE)
     SolverScalars *S;
     int coef_mode;
+    const DevAllreduce *dar = nullptr;  // kernel-side global sum (device pointer), nullptr: local only
+    int chan = 0;                       // its channel
 };
 
 // ----------------------------------------------------------------------------- kernels
@@ -177,6 +197,7 @@ struct DslashArgs {
     const void *clover;    // parity p: T (xpay) or T^{-1} (clover_inv)
     const void *ghost_back; // upper (non-dagger) half-spinors from rank-1, face layout
     const void *ghost_fwd;  // lower (non-dagger) half-spinors from rank+1
+    long ghost_rhs_bytes;   // multi-RHS halo: RHS k's ghost faces sit k * ghost_rhs_bytes further on
     // kernel-initiated halo: this launch consumes halo number s = *p2p_cseq + 1: before reading
     // ghosts its boundary CTAs wait until p2p_flags[0], p2p_flags[1] >= s (system-scope
     // acquire); ghosts of odd s sit p2p_pdist bytes on.  The launch's last CTA (counter

@@ -100,6 +100,43 @@ __device__ __forceinline__ void cta_sum_slots(const double *src, int b0, int b1,
         }
 }
 
+// Kernel-side global sum (DevAllreduce, internal.h) of the NRED totals in v, by one thread.
+__device__ __forceinline__ unsigned long long ld_acquire_sys_u64(const unsigned long long *p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ void st_release_sys_u64(unsigned long long *p, unsigned long long v) {
+    asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+template <int NRED>
+__device__ __forceinline__ void dev_allreduce(const DevAllreduce &d, int chan, double (&v)[NRED]) {
+    static_assert(NRED <= 3, "slot holds 3 sums");
+    const unsigned s = d.seq[chan] + 1u;
+    d.seq[chan] = s;
+    const size_t base = ((size_t)chan * 2 + (s & 1u)) * kMaxPeers;
+    for (int r = 0; r < d.nranks; ++r) {  // this rank's totals into slot [rank] of every rank
+        double *dst = d.slots[r] + (base + d.rank) * 4;
+        for (int k = 0; k < NRED; ++k) dst[k] = v[k];
+        st_release_sys_u64(reinterpret_cast<unsigned long long *>(dst + 3), (unsigned long long)s);
+    }
+    double tot[NRED];
+    for (int k = 0; k < NRED; ++k) tot[k] = 0.0;
+    const double *own = d.slots[d.rank];
+    for (int r = 0; r < d.nranks; ++r) {  // fixed rank order: bitwise identical on every rank
+        const double *src = own + (base + r) * 4;
+        const unsigned long long *sq = reinterpret_cast<const unsigned long long *>(src + 3);
+        bool ok = false;
+        for (long spin = 0; spin < (1L << 24) && !ok; ++spin) {
+            ok = ld_acquire_sys_u64(sq) == (unsigned long long)s;
+            if (!ok) __nanosleep(64);
+        }
+        if (!ok && d.err) atomicExch(d.err, 2);
+        for (int k = 0; k < NRED; ++k) tot[k] += *reinterpret_cast<const volatile double *>(src + k);
+    }
+    for (int k = 0; k < NRED; ++k) v[k] = tot[k];
+}
+
 // v[] -> this CTA's partial; the last CTA of the whole reduction produces t.out[0..NRED).
 // Layout: t.partials[0 .. total) CTA slots, then ceil(total/kGroup) group slots.
 // Counters: t.counter[0] groups done, t.counter[1 + g] CTAs done in group g (all zero on entry).
@@ -148,6 +185,7 @@ __device__ __forceinline__ void reduce_with_tail(double (&v)[NRED], const RedTai
     fence_acquire();
     cta_sum_slots<NRED, NT>(gslots, 0, ngroups, res, sm);
     if (threadIdx.x == 0) {
+        if (t.dar) dev_allreduce<NRED>(*t.dar, t.chan, res);  // the global sum, in-kernel
         for (int k = 0; k < NRED; ++k) t.out[k] = res[k];
         if (t.coef_mode != COEF_NONE) apply_coef(t.S, t.coef_mode);
         t.counter[0] = 0u;  // ready for the next stream-ordered reduction
