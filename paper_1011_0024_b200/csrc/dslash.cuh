@@ -505,6 +505,24 @@ __device__ __forceinline__ void pf_spinor_l1(const void *base, long stride, long
         for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + j)));
     }
 }
+// L1 prefetch of a site's clover (CLOVER_INV reads it only after the 8 hops): issued before the
+// temporal hops, the epilogue's streamed loads then hit L1 instead of paying a DRAM round trip
+// after the last hop.  QX_CLV_PF: 1 on (default for the pipelined half kernel), 0 off.
+#ifndef QX_CLV_PF
+#define QX_CLV_PF 1
+#endif
+template <int P>
+__device__ __forceinline__ void pf_clover_l1(const void *base, long stride, long i) {
+    if constexpr (P == 2) {
+#pragma unroll
+        for (int k = 0; k < 9; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + i)));
+        pf_l1(cptr(base, (size_t)144 * stride + 8 * i));
+    } else {
+        constexpr int NB = (P == 8) ? 36 : 18;
+#pragma unroll
+        for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + i)));
+    }
+}
 // one output site; red[] receives this site's contribution to the optional fused reduction
 // INMODE: load mode of the neighbour spinors (0 read-only path; 2 L2-coherent, for inputs
 // written by other CTAs earlier in the same launch — the fused Mhat kernel)
@@ -775,6 +793,9 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         comp_sp(A, I2{}, CF{});
         THop C, D;
         load_tf(C);
+#if QX_CLV_PF
+        if constexpr (KIND == QUDAX_CLOVER_INV || KIND == QUDAX_CLOVER_INV_XPAY) pf_clover_l1<P>(a.clover, a.stride, i);
+#endif
         comp_sp(B, I2{}, CB{});
         load_tb(D);
 #if QX_RED_PF

@@ -50,8 +50,11 @@ def main():
     ctx.gauge_load(U, K, CSW, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
     _, st = ctx.solve(b, tol=1e-10, delta=1e-2, maxiter=200, prec=8, prec_sloppy=4)
     print("nccl loopback", st["iters"], st["true_res"])
-    ctx.close()
-    print("sanitize workload done")
+    ctx.sync()
+    print("sanitize workload done", flush=True)
+    # leave without ncclCommDestroy: under compute-sanitizer NCCL's teardown did not return
+    # (r02a: every tool had finished the workload, reported nothing, then hung in close)
+    os._exit(0)
 
 
 if __name__ == "__main__":
