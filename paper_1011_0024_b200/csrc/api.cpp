@@ -509,35 +509,62 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         if (!red->S) global_sum(c, c->red_out, 3, red->res);
         else if (multi) device_sum_coef(c, red->S->red, 3, red->S, red->coef_mode);
     };
-    if (c->p2p.on) {  // kernel-initiated halo over peer memory (QUDAX_HALO_P2P), T-only split
+    if (c->p2p.on) {  // kernel-initiated halo over peer memory (QUDAX_HALO_P2P), any process grid
         auto &q = c->p2p;
         const int pi = prec_idx(prec);
-        args.ghosted = 1;
-        args.ghost_back = q.base + q.off_gb[pi];
-        args.ghost_fwd = q.base + q.off_gf[pi];
+        args.ghosted = (g.split >> 3) & 1;
+        args.ghost_back = q.base + q.off_g[pi][3][0];
+        args.ghost_fwd = q.base + q.off_g[pi][3][1];
+        args.p2p_pdist = (long)q.pdist[pi][3];
+        for (int m = 0; m < 3; ++m) {
+            args.sghost_back[m] = q.base + q.off_g[pi][m][0];
+            args.sghost_fwd[m] = q.base + q.off_g[pi][m][1];
+            args.sp2p_pdist[m] = (long)q.pdist[pi][m];
+        }
         args.p2p_cseq = reinterpret_cast<unsigned *>(q.base + q.off_cseq);
         args.p2p_ccount = reinterpret_cast<unsigned *>(q.base + q.off_ccount);
-        args.p2p_pdist = (long)q.pdist[pi];
+        args.p2p_mask = g.split;
         unsigned *own_flags = reinterpret_cast<unsigned *>(q.base + q.off_flags);
-        // our t=0 face -> rank-1's ghost_fwd (its flags[1]); t=T_loc-1 face -> rank+1's ghost_back (flags[0])
+        // our x_mu = 0 face -> the backward neighbour's FORWARD ghost (its flag 2 mu + 1); our
+        // x_mu = L-1 face -> the forward neighbour's BACKWARD ghost (its flag 2 mu)
+        P2PPackArgs pk{};
+        pk.mask = g.split;
+        pk.q = 1 - p;
+        pk.stride = g.stride;
+        for (int m = 0; m < 4; ++m) {
+            pk.L[m] = g.L[m];
+            pk.Fd[m] = g.Fd[m];
+            pk.fsd[m] = g.fsd[m];
+            if (!(g.split >> m & 1)) continue;
+            pk.dst_b[m] = q.peer_b[m] + q.off_g[pi][m][1];
+            pk.dst_f[m] = q.peer_f[m] + q.off_g[pi][m][0];
+            pk.pdist[m] = (long)q.pdist[pi][m];
+            pk.flag_b[m] = reinterpret_cast<unsigned *>(q.peer_b[m] + q.off_flags) + 2 * m + 1;
+            pk.flag_f[m] = reinterpret_cast<unsigned *>(q.peer_f[m] + q.off_flags) + 2 * m;
+        }
+        pk.seq = reinterpret_cast<unsigned *>(q.base + q.off_seq);
+        pk.count = reinterpret_cast<unsigned *>(q.base + q.off_count);
+        pk.halt = c->halt;
+        pk.half_back = dagger ? 0 : 1;  // non-dagger: lower spins go backward (reading Q15)
+        pk.half_fwd = dagger ? 1 : 0;
         auto pack = [&](cudaStream_t st) {
-            launch_pack_faces_p2p(prec, dagger, g, in, q.peer_back + q.off_gf[pi], q.peer_fwd + q.off_gb[pi],
-                                  q.pdist[pi], reinterpret_cast<unsigned *>(q.peer_back + q.off_flags) + 1,
-                                  reinterpret_cast<unsigned *>(q.peer_fwd + q.off_flags),
-                                  reinterpret_cast<unsigned *>(q.base + q.off_seq),
-                                  reinterpret_cast<unsigned *>(q.base + q.off_count), c->halt, st);
+            launch_pack_p2p(prec, dagger, pk, in, st);
             c->launches += 1;
         };
-        if (c->overlap && g.T_loc > 2) {
+        const bool sp = spatial_split(g) != 0;
+        const bool tail = c->overlap && (sp || g.T_loc > 2);
+        if (tail) {
             // ONE Dslash launch (RANGE_TAIL) beside the pack on the high-priority comm stream:
-            // interior CTAs first, the boundary CTAs at the grid's tail acquire the neighbours'
-            // flags.  The join after it only keeps `in` alive until our own pack has read it.
+            // interior sites first (T-only: t in [1, T_loc-2]; a grid: the interior box), the
+            // boundary CTAs at the grid's tail acquire the neighbours' flags.  The join after it
+            // only keeps `in` alive until our own pack has read it.
             QX_CUDA(cudaEventRecord(c->ev_in, c->stream));
             QX_CUDA(cudaStreamWaitEvent(c->comm_stream, c->ev_in, 0));
             pack(c->comm_stream);
             QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
             args.p2p_flags = own_flags;
             args.reverse = 0;  // the waiting CTAs must be the last ones
+            args.tail_ni = sp ? (int)g.n_int : (int)((g.T_loc - 2) * g.F);
             launch(RANGE_TAIL, (int)g.Vh);
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
         } else {
@@ -1190,11 +1217,14 @@ static void setup_p2p(qudax_ctx *c) {
     const int precs[3] = {8, 4, 2};
     for (int k = 0; k < 3; ++k) {
         const int pi = prec_idx(precs[k]);
-        q.pdist[pi] = up(face_bytes(precs[k], g.fstride));
-        q.off_gb[pi] = cur;
-        cur += 2 * q.pdist[pi];
-        q.off_gf[pi] = cur;
-        cur += 2 * q.pdist[pi];
+        for (int m = 0; m < 4; ++m) {  // ghosts of every split dimension, two sequence parities each
+            if (!(g.split >> m & 1)) continue;
+            q.pdist[pi][m] = up(m == 3 ? face_bytes(precs[k], g.fstride) : sface_bytes(precs[k], m, g.fsd[m]));
+            q.off_g[pi][m][0] = cur;
+            cur += 2 * q.pdist[pi][m];
+            q.off_g[pi][m][1] = cur;
+            cur += 2 * q.pdist[pi][m];
+        }
     }
     q.off_flags = cur;
     q.off_seq = cur + 64;
@@ -1222,8 +1252,13 @@ static void setup_p2p(qudax_ctx *c) {
         allgather_small(c, &mine, sizeof(Rec), all.data());
         const bool map_all = g.nranks <= kMaxPeers;
         q.opened.assign(g.nranks, nullptr);
+        auto is_nb = [&](int r) {
+            for (int m = 0; m < 4; ++m)
+                if ((g.split >> m & 1) && (r == g.nbf[m] || r == g.nbb[m])) return true;
+            return false;
+        };
         for (int r = 0; r < g.nranks; ++r) {
-            if (r == g.rank || !(map_all || r == g.nbf[3] || r == g.nbb[3])) continue;
+            if (r == g.rank || !(map_all || is_nb(r))) continue;
             const Rec &rec = all[r];
             if (std::strncmp(rec.bus, mine.bus, sizeof(mine.bus)) != 0) {  // another GPU (else test mode)
                 int peer = -1, can = 0;
@@ -1242,12 +1277,14 @@ static void setup_p2p(qudax_ctx *c) {
             q.opened[r] = static_cast<char *>(pr);
         }
         auto region = [&](int r) { return r == g.rank ? q.base : q.opened[r]; };
-        q.peer_back = region(g.nbb[3]);
-        q.peer_fwd = region(g.nbf[3]);
+        for (int m = 0; m < 4; ++m) {
+            q.peer_b[m] = region(g.nbb[m]);
+            q.peer_f[m] = region(g.nbf[m]);
+        }
         if (map_all)
             for (int r = 0; r < g.nranks; ++r) q.peer[r] = region(r);
     } else {  // loopback: the neighbour is this rank
-        q.peer_back = q.peer_fwd = q.base;
+        for (int m = 0; m < 4; ++m) q.peer_b[m] = q.peer_f[m] = q.base;
         q.peer[0] = q.base;
     }
     // kernel-side allreduce descriptor (device memory), when every rank is mapped
@@ -1276,8 +1313,6 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
     if (p->comm == QUDAX_COMM_NONE && p->nranks != 1) return QUDAX_ERR_ARG;
     if (p->comm == QUDAX_COMM_NCCL && !p->nccl_id) return QUDAX_ERR_ARG;
     if (p->comm == QUDAX_COMM_HOST && (!p->host_exchange || !p->host_allreduce)) return QUDAX_ERR_ARG;
-    // the kernel-initiated halo covers the T faces; the comm halo every dimension
-    if (p->halo == QUDAX_HALO_P2P && part.split_mask != 8) return QUDAX_ERR_UNSUPPORTED;
     // a loopback dimension without a transport has nobody to move its faces
     if (p->comm == QUDAX_COMM_NONE && p->halo != QUDAX_HALO_P2P && part.split_mask) return QUDAX_ERR_ARG;
     auto *c = new qudax_ctx();

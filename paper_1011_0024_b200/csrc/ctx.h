@@ -104,17 +104,19 @@ struct qudax_ctx {
     int *blist = nullptr;  // boundary sites (complement of the interior box) when X/Y/Z is split
 
     // kernel-initiated halo over peer memory (QUDAX_HALO_P2P).  One cudaMalloc region per rank,
-    // identical layout on every rank: per precision ghost_back[2], ghost_fwd[2] (sequence
-    // parity), then flags[2] (flags[0] raised by rank-1 after it filled ghost_back, flags[1] by
-    // rank+1 after ghost_fwd), the producer (pack) and consumer (Dslash) halo counters and
-    // their CTA counters.
+    // identical layout on every rank: per precision and split dimension mu ghost_back[2],
+    // ghost_fwd[2] (sequence parity), then flags[4][2] (flags[mu][0] raised by the backward
+    // neighbour along mu after it filled ghost_back, flags[mu][1] by the forward one after
+    // ghost_fwd), the producer (pack) and consumer (Dslash) halo counters and their CTA
+    // counters, and the kernel-side allreduce slots.
     struct P2P {
         bool on = false;
         char *base = nullptr;                       // own region (cudaMalloc, IPC-exported)
-        char *peer_back = nullptr, *peer_fwd = nullptr;  // neighbours' regions (IPC-mapped or own)
+        char *peer_b[4] = {}, *peer_f[4] = {};           // neighbours' regions per dimension (IPC-mapped or own)
         char *peer[qx::kMaxPeers] = {};                  // every rank's region (nranks <= kMaxPeers)
         std::vector<char *> opened;                      // IPC mappings to close at finalize
-        size_t off_gb[3] = {}, off_gf[3] = {}, pdist[3] = {};
+        // per precision and split dimension: ghost_back / ghost_fwd (x2 sequence parities)
+        size_t off_g[3][4][2] = {}, pdist[3][4] = {};
         size_t off_flags = 0, off_seq = 0, off_count = 0, off_cseq = 0, off_ccount = 0, off_ar = 0, bytes = 0;
     } p2p;
     // kernel-side allreduce descriptor (device memory) of the P2P mode, nullptr otherwise

@@ -530,12 +530,16 @@ __device__ __forceinline__ void pf_clover_l1(const void *base, long stride, long
 // separate instantiation so the unpartitioned kernels keep their register allocation
 template <int P, int RECON, bool DAG, int KIND, int INMODE = 0, bool SS = false>
 __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin, void *fout, const void *fx, int tid,
-                                            double red[3], long goff = 0) {
+                                            double red[3], long goff = 0, int sbit = 0) {
     using R = typename Prec<P>::R;
     if (a.reverse) tid = a.nthreads - 1 - tid;
     const int X = a.X, Y = a.Y, Z = a.Z, Xh = a.Xh;
     int i, xh, y, z, t;
-    if (SS && a.range == RANGE_INTERIOR) {  // the interior box of a multi-dimensional split
+    // the boundary sites of a multi-dimensional split follow the interior box in one RANGE_TAIL
+    // launch (kernel-initiated halo)
+    const bool ss_box = SS && (a.range == RANGE_INTERIOR || (a.range == RANGE_TAIL && tid < a.tail_ni));
+    if (SS && a.range == RANGE_TAIL && !ss_box) tid -= a.tail_ni;
+    if (ss_box) {  // the interior box of a multi-dimensional split
         int r = tid;
         xh = r % a.bn[0] + a.blo[0];
         r /= a.bn[0];
@@ -547,12 +551,12 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     } else {
         if (a.range == RANGE_ALL) i = tid;
         else if (a.range == RANGE_INTERIOR) i = a.F + tid;  // T-only split: t in [1, T_loc-2]
+        else if (SS) i = __ldg(a.blist + tid);  // complement of the interior box (BOUNDARY / TAIL)
         else if (a.range == RANGE_TAIL) {
             const int ni = (a.T_loc - 2) * a.F;
             const int j = tid - ni;
             i = (tid < ni) ? a.F + tid : ((j < a.F) ? j : (a.T_loc - 1) * a.F + (j - a.F));
-        } else if (SS) i = __ldg(a.blist + tid);  // complement of the interior box
-        else i = (tid < a.F) ? tid : (a.T_loc - 1) * a.F + (tid - a.F);
+        } else i = (tid < a.F) ? tid : (a.T_loc - 1) * a.F + (tid - a.F);
         int r = fdiv(i, a.dXh);
         xh = i - r * Xh;
         const int r2 = fdiv(r, a.dY);
@@ -608,9 +612,9 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         if constexpr (SS && MU == 0) {
             if (a.smask & 1) {
                 const int f = face_index<0>(x, y, z, t, X, Y, Z);
-                if (coord == Lmu - 1) { fsrc = a.sghost_fwd[0]; fstr = a.sfs[0]; nf = f; }
+                if (coord == Lmu - 1) { fsrc = cptr(a.sghost_fwd[0], sbit ? a.sp2p_pdist[0] : 0); fstr = a.sfs[0]; nf = f; }
                 if (coord == 0) {
-                    bsrc = a.sghost_back[0]; bstr = a.sfs[0]; nb = f;
+                    bsrc = cptr(a.sghost_back[0], sbit ? a.sp2p_pdist[0] : 0); bstr = a.sfs[0]; nb = f;
                     lbsrc = a.gauge_sghost[0]; lbstr = a.sfs[0]; lbi = f;
                 }
             }
@@ -624,7 +628,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
                 Cx<R> h0[3], h1[3], u[3][3];
                 R sc;
                 if (gf) {
-                    sc = ghost_half<P, MU, SF, DF>(a.sghost_fwd[MU], a.sfs[MU], f, h0, h1);
+                    sc = ghost_half<P, MU, SF, DF>(cptr(a.sghost_fwd[MU], sbit ? a.sp2p_pdist[MU] : 0), a.sfs[MU], f, h0, h1);
                 } else {
                     RawVec<P, 24> sv;
                     sv.template load_spinor<INMODE>(fin, a.stride, nf);
@@ -641,7 +645,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
                 }
                 spatial_mult_expand<MU, SF, false, DF>(h0, h1, u, acc, sc);
                 if (gb) {
-                    sc = ghost_half<P, MU, SB, DF>(a.sghost_back[MU], a.sfs[MU], f, h0, h1);
+                    sc = ghost_half<P, MU, SB, DF>(cptr(a.sghost_back[MU], sbit ? a.sp2p_pdist[MU] : 0), a.sfs[MU], f, h0, h1);
                     RawLink<P, RECON> l;
                     l.load(a.gauge_sghost[MU], a.sfs[MU], f);
                     sc *= dec_link<DF>(l, u);
@@ -955,20 +959,24 @@ __device__ __forceinline__ unsigned ld_acquire_sys(const unsigned *p) {
     asm volatile("ld.acquire.sys.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
     return v;
 }
-__device__ __forceinline__ long p2p_wait(const DslashArgs &a) {
+__device__ __forceinline__ int p2p_wait(const DslashArgs &a) {
     __shared__ unsigned s_seq;
     if (threadIdx.x == 0) {
         const unsigned s = *reinterpret_cast<const volatile unsigned *>(a.p2p_cseq) + 1u;
         bool ok = false;
         for (long spin = 0; spin < (1L << 24) && !ok; ++spin) {  // >= 2 s of 128 ns sleeps
-            ok = (int)(ld_acquire_sys(a.p2p_flags) - s) >= 0 && (int)(ld_acquire_sys(a.p2p_flags + 1) - s) >= 0;
+            ok = true;
+            for (int m = 0; m < 4 && ok; ++m)
+                if (a.p2p_mask >> m & 1)
+                    ok = (int)(ld_acquire_sys(a.p2p_flags + 2 * m) - s) >= 0 &&
+                         (int)(ld_acquire_sys(a.p2p_flags + 2 * m + 1) - s) >= 0;
             if (!ok) __nanosleep(128);
         }
         if (!ok && a.err) atomicExch(a.err, 1);
         s_seq = s;
     }
     __syncthreads();
-    return (s_seq & 1u) ? a.p2p_pdist : 0L;
+    return (int)(s_seq & 1u);
 }
 
 template <int P, int RECON, bool DAG, int KIND, bool SS>
@@ -989,9 +997,13 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     void *fout = a.nrhs > 1 ? a.out_m[rhs] : a.out;
     const void *fx = a.nrhs > 1 ? a.x_m[rhs] : a.x;
     long goff = (long)rhs * a.ghost_rhs_bytes;  // multi-RHS halo: this RHS's ghost faces
+    int sbit = 0;                               // kernel-initiated halo: sequence parity of the ghosts
     // RANGE_TAIL: only CTAs holding boundary sites (the grid's last ones) wait for the halo
-    if (a.p2p_flags && (a.range != RANGE_TAIL || (blk + 1) * (int)blockDim.x > (a.T_loc - 2) * a.F)) goff = p2p_wait(a);
-    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND, 0, SS>(a, fin, fout, fx, tid, red, goff);
+    if (a.p2p_flags && (a.range != RANGE_TAIL || (blk + 1) * (int)blockDim.x > a.tail_ni)) {
+        sbit = p2p_wait(a);
+        goff = sbit ? a.p2p_pdist : 0L;
+    }
+    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND, 0, SS>(a, fin, fout, fx, tid, red, goff, sbit);
     if (a.p2p_flags) {  // the last CTA to finish advances the consumed-halo counter
         __syncthreads();
         if (threadIdx.x == 0 && atomicAdd(a.p2p_ccount, 1u) == gridDim.x - 1) {

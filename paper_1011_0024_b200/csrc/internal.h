@@ -199,14 +199,19 @@ struct DslashArgs {
     const void *ghost_fwd;  // lower (non-dagger) half-spinors from rank+1
     long ghost_rhs_bytes;   // multi-RHS halo: RHS k's ghost faces sit k * ghost_rhs_bytes further on
     // kernel-initiated halo: this launch consumes halo number s = *p2p_cseq + 1: before reading
-    // ghosts its boundary CTAs wait until p2p_flags[0], p2p_flags[1] >= s (system-scope
-    // acquire); ghosts of odd s sit p2p_pdist bytes on.  The launch's last CTA (counter
+    // ghosts its boundary CTAs wait until p2p_flags[2 mu], p2p_flags[2 mu + 1] >= s for every
+    // split dimension mu of p2p_mask (system-scope acquire); ghosts of odd s sit p2p_pdist (T)
+    // / sp2p_pdist[mu] (X, Y, Z) bytes on.  RANGE_TAIL: the first tail_ni sites are interior
+    // (no ghost reads), the CTAs beyond them wait.  The launch's last CTA (counter
     // p2p_ccount) advances *p2p_cseq.  The pack kernel keeps its own producer counter, so the
     // two may run concurrently.
     unsigned *p2p_cseq;
     unsigned *p2p_ccount;
     const unsigned *p2p_flags;
     long p2p_pdist;
+    long sp2p_pdist[3];
+    int p2p_mask;
+    int tail_ni;
     // optional fused reduction over the output (BiCGstab, P:542-558 kernel fusion)
     int red_kind;          // RED_NONE, RED_XDOT_NORM: (<out,x>, |out|^2), RED_RHAT_DOT: <rhat,out>
     RedTail tail;          // 3 sums per CTA; block_offset set per launch (split launches)
@@ -251,13 +256,25 @@ size_t sface_bytes(int prec, int mu, long fs);
 // (upper if !dagger) -> send_fwd.  `in` is the Dslash input field (parity 1-p).
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back,
                        void *send_fwd, const int *halt, cudaStream_t s);
-// kernel-initiated halo (QUDAX_HALO_P2P): the same faces stored straight into the neighbours'
-// ghost buffers dst_back / dst_fwd (+ pdist bytes for odd sequence numbers), then flag_back /
-// flag_fwd (in the neighbours' memory) set to the new sequence number with a system-scope
-// release.  seq / count: this rank's sequence counter and CTA counter (device).
-void launch_pack_faces_p2p(int prec, int dagger, const Geom &g, const void *in, char *dst_back, char *dst_fwd,
-                           size_t pdist, unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count,
-                           const int *halt, cudaStream_t s);
+
+// kernel-initiated halo of any process grid (QUDAX_HALO_P2P): all split dimensions' faces
+// stored into the neighbours' ghosts (peer memory), then their flags raised (layout.cu)
+struct P2PPackArgs {
+    int L[4];
+    int mask;               // split dimensions
+    int q;                  // parity of the packed (input) field
+    long Fd[4], fsd[4];     // per-parity face sites along mu, padded
+    long stride;
+    char *dst_b[4];         // backward neighbour's forward-ghost buffer (sequence parity 0)
+    char *dst_f[4];         // forward neighbour's backward-ghost buffer
+    long pdist[4];          // bytes to the sequence-parity-1 buffer
+    unsigned *flag_b[4];    // backward neighbour's "forward ghost filled" flag of mu
+    unsigned *flag_f[4];    // forward neighbour's "backward ghost filled" flag of mu
+    unsigned *seq, *count;  // this rank's producer sequence and CTA counter
+    const int *halt;
+    int half_back, half_fwd; // T faces: spin halves sent backward / forward (reading Q15)
+};
+void launch_pack_p2p(int prec, int dagger, const P2PPackArgs &a, const void *in, cudaStream_t s);
 
 // layout conversion (DR AoS fp64 <-> NR SoA prec), one parity
 void launch_spinor_import(int prec, const Geom &g, int parity, const double *src, void *dst, cudaStream_t s);

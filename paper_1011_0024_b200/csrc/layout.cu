@@ -591,56 +591,12 @@ __global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int 
     k_pack_faces_body<P>(F, T_loc, stride, fstride, half_back, half_fwd, in, sb, sf);
 }
 
-// Kernel-initiated halo: k_pack_faces storing into the neighbours' ghosts (peer memory), then
-// the last CTA raises the neighbours' flags.  Each CTA's stores are ordered before its arrival
-// on the counter by bar.sync + one system-scope fence (cumulative, as in a grid barrier), and
-// the last CTA's fence + release orders all of them before the flags.
+// system-scope release store of a flag (the kernel-initiated halo's sequence numbers): each CTA's
+// ghost stores are ordered before its arrival on the pack counter by bar.sync + one system-scope
+// fence (cumulative, as in a grid barrier), and the last CTA's fence + release orders all of
+// them before the flags
 __device__ __forceinline__ void st_release_sys(unsigned *p, unsigned v) {
     asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
-}
-template <int P>
-__global__ void k_pack_faces_p2p(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
-                                 const void *__restrict__ in, char *dst_back, char *dst_fwd, long pdist,
-                                 unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count,
-                                 const int *halt) {
-    __shared__ bool last;
-    // a halted solver iteration (every rank halts the same one: the decision is taken on
-    // globally summed scalars) skips both the pack and the consuming Dslash, so producer and
-    // consumer sequence counters stay in step
-    if (halted(halt)) return;
-    const unsigned s = *reinterpret_cast<volatile unsigned *>(seq) + 1u;
-    const long off = (s & 1u) ? pdist : 0L;
-    k_pack_faces_body<P>(F, T_loc, stride, fstride, half_back, half_fwd, in, dst_back + off, dst_fwd + off);
-    __syncthreads();
-    if (threadIdx.x == 0) {
-        __threadfence_system();
-        last = (atomicAdd(count, 1u) == gridDim.x - 1);
-    }
-    __syncthreads();
-    if (last && threadIdx.x == 0) {
-        *count = 0u;
-        *seq = s;
-        __threadfence_system();
-        st_release_sys(flag_back, s);
-        st_release_sys(flag_fwd, s);
-    }
-}
-
-void launch_pack_faces_p2p(int prec, int dagger, const Geom &g, const void *in, char *dst_back, char *dst_fwd,
-                           size_t pdist, unsigned *flag_back, unsigned *flag_fwd, unsigned *seq, unsigned *count,
-                           const int *halt, cudaStream_t s) {
-    const int half_back = dagger ? 0 : 1;
-    const int half_fwd = dagger ? 1 : 0;
-    const int T = 128;
-    const int b = nblk(2 * g.F, T);
-#define QX_PP(P)                                                                                                \
-    k_pack_faces_p2p<P><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, dst_back,   \
-                                        dst_fwd, (long)pdist, flag_back, flag_fwd, seq, count, halt)
-    if (prec == 8) QX_PP(8);
-    else if (prec == 4) QX_PP(4);
-    else QX_PP(2);
-#undef QX_PP
-    QX_CUDA(cudaGetLastError());
 }
 
 // Faces of the partitioned X / Y / Z: the x_mu = 0 face goes backward and
@@ -661,43 +617,34 @@ struct SPackArgs {
     void *sb[3], *sf[3];
     const int *halt;
 };
+// one face site of a partitioned X / Y / Z (face index f of dimension mu, fwd: the x_mu = L-1
+// face) -> dst (face layout, fs padded sites)
 template <int P, bool DAG>
-__global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *__restrict__ in) {
+__device__ __forceinline__ void pack_spatial_one(int mu, long f, bool fwd, const int L[4], int q, long stride,
+                                                 const void *__restrict__ in, void *dst, long fs) {
     using R = typename Prec<P>::R;
-    if (halted(a.halt)) return;
-    long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
-    int mu = 0;
-    for (; mu < 3; ++mu) {
-        if (!(a.mask >> mu & 1)) continue;
-        if (k < 2 * a.Fd[mu]) break;
-        k -= 2 * a.Fd[mu];
-    }
-    if (mu == 3) return;
-    const bool fwd = k >= a.Fd[mu];
-    const long f = fwd ? k - a.Fd[mu] : k;
     int c[4];
-    face_site(mu, f, fwd ? a.L[mu] - 1 : 0, a.q, a.L, c);
-    const long i = (((long)(c[3] * a.L[2] + c[2]) * a.L[1] + c[1]) * a.L[0] + c[0]) >> 1;
-    void *dst = fwd ? a.sf[mu] : a.sb[mu];
+    face_site(mu, f, fwd ? L[mu] - 1 : 0, q, L, c);
+    const long i = (((long)(c[3] * L[2] + c[2]) * L[1] + c[1]) * L[0] + c[0]) >> 1;
     if (sface_raw(P, mu)) {  // the raw record (+ half norm): bits only, the receiver projects
         if constexpr (P == 2) {
             for (int hf = 0; hf < 2; ++hf) {
-                reinterpret_cast<uint4 *>(mptr(dst, h_spinor_u(a.fsd[mu], hf)))[f] =
-                    reinterpret_cast<const uint4 *>(cptr(in, h_spinor_u(a.stride, hf)))[i];
-                reinterpret_cast<uint2 *>(mptr(dst, h_spinor_v(a.fsd[mu], hf)))[f] =
-                    reinterpret_cast<const uint2 *>(cptr(in, h_spinor_v(a.stride, hf)))[i];
+                reinterpret_cast<uint4 *>(mptr(dst, h_spinor_u(fs, hf)))[f] =
+                    reinterpret_cast<const uint4 *>(cptr(in, h_spinor_u(stride, hf)))[i];
+                reinterpret_cast<uint2 *>(mptr(dst, h_spinor_v(fs, hf)))[f] =
+                    reinterpret_cast<const uint2 *>(cptr(in, h_spinor_v(stride, hf)))[i];
             }
-            SpinorIO<2>::norms(dst, a.fsd[mu])[f] = SpinorIO<2>::norms(in, a.stride)[i];
+            SpinorIO<2>::norms(dst, fs)[f] = SpinorIO<2>::norms(in, stride)[i];
         } else {
             using V = typename StoreVec<P>::V;
             constexpr int NB = (P == 8) ? 12 : 6;
             for (int b = 0; b < NB; ++b)
-                reinterpret_cast<V *>(dst)[b * a.fsd[mu] + f] = reinterpret_cast<const V *>(in)[b * a.stride + i];
+                reinterpret_cast<V *>(dst)[b * fs + f] = reinterpret_cast<const V *>(in)[b * stride + i];
         }
         return;
     }
     RawVec<P, 24> raw;
-    raw.template load_spinor<0>(in, a.stride, i);
+    raw.template load_spinor<0>(in, stride, i);
     R v[24];
     Cx<R> ps[4][3], h0[3], h1[3];
     raw.decode(v);
@@ -710,7 +657,102 @@ __global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *
     } else {
         if (fwd) spatial_project<2, SB>(ps, h0, h1); else spatial_project<2, SF>(ps, h0, h1);
     }
-    SFace<R>::store(dst, a.fsd[mu], f, h0, h1);
+    SFace<R>::store(dst, fs, f, h0, h1);
+}
+
+template <int P, bool DAG>
+__global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *__restrict__ in) {
+    if (halted(a.halt)) return;
+    long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    int mu = 0;
+    for (; mu < 3; ++mu) {
+        if (!(a.mask >> mu & 1)) continue;
+        if (k < 2 * a.Fd[mu]) break;
+        k -= 2 * a.Fd[mu];
+    }
+    if (mu == 3) return;
+    const bool fwd = k >= a.Fd[mu];
+    const long f = fwd ? k - a.Fd[mu] : k;
+    pack_spatial_one<P, DAG>(mu, f, fwd, a.L, a.q, a.stride, in, fwd ? a.sf[mu] : a.sb[mu], a.fsd[mu]);
+}
+
+// Kernel-initiated halo of a general process grid (QUDAX_HALO_P2P): every
+// split dimension's two faces (T: the diagonal-projector halves, bits only; X / Y / Z: as
+// k_pack_spatial) stored straight into the neighbours' ghost buffers (peer memory), then the
+// last CTA raises, in each neighbour, the flag of the ghost it filled (system-scope release of
+// the sequence number).  One launch for all dimensions: one producer counter.
+template <int P, bool DAG>
+__global__ void k_pack_p2p(const __grid_constant__ P2PPackArgs a, const void *__restrict__ in) {
+    __shared__ bool last;
+    if (halted(a.halt)) return;
+    const unsigned s = *reinterpret_cast<volatile unsigned *>(a.seq) + 1u;
+    const bool odd = (s & 1u) != 0;
+    long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    int mu = 0;
+    for (; mu < 4; ++mu) {
+        if (!(a.mask >> mu & 1)) continue;
+        if (k < 2 * a.Fd[mu]) break;
+        k -= 2 * a.Fd[mu];
+    }
+    if (mu < 4) {
+        const bool fwd = k >= a.Fd[mu];
+        const long f = fwd ? k - a.Fd[mu] : k;
+        char *dst = (fwd ? a.dst_f[mu] : a.dst_b[mu]) + (odd ? a.pdist[mu] : 0);
+        if (mu == 3) {
+            const long i = fwd ? (a.L[3] - 1) * a.Fd[3] + f : f;
+            const int half = fwd ? a.half_fwd : a.half_back;
+            if constexpr (P == 8) {
+                const double2 *sp = reinterpret_cast<const double2 *>(in);
+                double2 *d = reinterpret_cast<double2 *>(dst);
+                for (int b = 0; b < 6; ++b) d[b * a.fsd[3] + f] = sp[(6 * half + b) * a.stride + i];
+            } else if constexpr (P == 4) {
+                const float4 *sp = reinterpret_cast<const float4 *>(in);
+                float4 *d = reinterpret_cast<float4 *>(dst);
+                for (int b = 0; b < 3; ++b) d[b * a.fsd[3] + f] = sp[(3 * half + b) * a.stride + i];
+            } else {
+                reinterpret_cast<uint4 *>(dst)[f] = reinterpret_cast<const uint4 *>(cptr(in, h_spinor_u(a.stride, half)))[i];
+                reinterpret_cast<uint2 *>(mptr(dst, (size_t)16 * a.fsd[3]))[f] =
+                    reinterpret_cast<const uint2 *>(cptr(in, h_spinor_v(a.stride, half)))[i];
+                FaceIO<2>::norms(dst, a.fsd[3])[f] = SpinorIO<2>::norms(in, a.stride)[i];
+            }
+        } else {
+            pack_spatial_one<P, DAG>(mu, f, fwd, a.L, a.q, a.stride, in, dst, a.fsd[mu]);
+        }
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence_system();
+        last = (atomicAdd(a.count, 1u) == gridDim.x - 1);
+    }
+    __syncthreads();
+    if (last && threadIdx.x == 0) {
+        *a.count = 0u;
+        *a.seq = s;
+        __threadfence_system();
+        for (int m = 0; m < 4; ++m) {
+            if (!(a.mask >> m & 1)) continue;
+            st_release_sys(a.flag_b[m], s);  // the backward neighbour's "forward ghost filled"
+            st_release_sys(a.flag_f[m], s);  // the forward neighbour's "backward ghost filled"
+        }
+    }
+}
+
+void launch_pack_p2p(int prec, int dagger, const P2PPackArgs &a, const void *in, cudaStream_t s) {
+    long n = 0;
+    for (int m = 0; m < 4; ++m)
+        if (a.mask >> m & 1) n += 2 * a.Fd[m];
+    const int T = 128;
+    const int b = n > 0 ? nblk(n, T) : 1;
+#define QX_PP2(PP)                                                                  \
+    if (prec == PP) {                                                               \
+        if (dagger) k_pack_p2p<PP, true><<<b, T, 0, s>>>(a, in);                     \
+        else k_pack_p2p<PP, false><<<b, T, 0, s>>>(a, in);                           \
+        QX_CUDA(cudaGetLastError());                                                 \
+        return;                                                                      \
+    }
+    QX_PP2(8) QX_PP2(4) QX_PP2(2)
+#undef QX_PP2
+    throw Error(QUDAX_ERR_ARG, "pack p2p: bad precision");
 }
 
 size_t sface_bytes(int prec, int mu, long fs) { return sface_raw(prec, mu) ? spinor_bytes(prec, fs) : (size_t)12 * prec * fs; }

@@ -94,10 +94,67 @@ def test_loopback_split_dims_bitwise(torch_cuda, prec, mask):
     loop.close()
 
 
-def test_p2p_rejects_spatial_split(torch_cuda):
-    with pytest.raises(qudax.QudaxError) as e:
-        qudax.Context((8, 4, 6, 8), halo=qudax.HALO_P2P, split_mask=0b1100)
-    assert e.value.status == 5
+@pytest.mark.parametrize("mask", [0b0100, 0b1100, 0b0001, 0b1111])
+@pytest.mark.parametrize("prec", [8, 4, 2])
+@pytest.mark.parametrize("overlap", [True, False])
+def test_p2p_split_dims_bitwise(torch_cuda, prec, mask, overlap):
+    """Kernel-initiated halo of a multi-dimensional split (SURVEY 8(f) item 1 for X / Y / Z
+    faces), loopback at N = 1: ONE pack kernel stores every split dimension's faces into the
+    (own) ghost buffers and raises the per-dimension flags; ONE Dslash launch runs the interior
+    box first and the boundary list in the CTAs that acquire the flags (overlap), or waits in
+    every CTA (no overlap).  Bitwise = unsplit for every precision, kind, parity and dagger."""
+    dims = (8, 4, 6, 8)
+    U = qgen.gauge(dims, 1241)
+    psi = qgen.spinor(dims, 1242)
+    x = qgen.spinor(dims, 1243)
+    ref = qudax.Context(dims)
+    loop = qudax.Context(dims, halo=qudax.HALO_P2P, split_mask=mask, overlap=overlap)
+    assert loop.partition["split_mask"] == mask
+    outs = {}
+    for name, c in (("ref", ref), ("loop", loop)):
+        c.gauge_load(U, 0.12, 1.0, prec=prec, recon=12)
+        fi, fo, fx = c.new_field(prec), c.new_field(prec), c.new_field(prec)
+        res = []
+        for p in (0, 1):
+            c.spinor_load(fi, prec, 1 - p, psi)
+            c.spinor_load(fx, prec, p, x)
+            for dagger in (False, True):
+                for kind in (0, 1, 2, 3):
+                    c.dslash(fo, fi, prec, p, dagger=dagger, kind=kind, x=fx, a=-0.2)
+                    c.sync()
+                    res.append(fo.cpu().numpy().copy())
+        fa, fb, fc = c.new_field(prec), c.new_field(prec), c.new_field(prec)
+        c.spinor_load(fa, prec, 0, psi)
+        c.matpc(fb, fa, prec)
+        c.matpc(fc, fb, prec, dagger=True)
+        c.mdagm(fb, fc, prec)
+        c.sync()
+        res.append(fb.cpu().numpy().copy())
+        outs[name] = res
+    for k, (a, b) in enumerate(zip(outs["ref"], outs["loop"])):
+        assert np.array_equal(a, b), k
+    ref.close()
+    loop.close()
+
+
+def test_p2p_split_dims_solve(torch_cuda):
+    """Mixed-precision solve with Y, Z and T split through the kernel-initiated halo and the
+    kernel-side allreduce (loopback, graph replay): the unsplit solve's iterations and solution
+    (fp32 sloppy: the fused reductions' fp64 sums of fp32 site partials are exact, so the
+    different CTA grouping of the tail launch does not change them)."""
+    dims = (8, 4, 4, 16)
+    U = qgen.gauge(dims, 1251, eps=0.1)
+    b = qgen.point_source(dims, 0, 2)
+    res = {}
+    for name, kw in (("ref", {}), ("p2p", {"halo": qudax.HALO_P2P, "split_mask": 0b1110})):
+        c = qudax.Context(dims, **kw)
+        c.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+        x, st = c.solve(b, tol=1e-12, delta=0.1, maxiter=1000, prec=8, prec_sloppy=4)
+        res[name] = (x, st)
+        c.close()
+    assert res["ref"][1]["iters"] == res["p2p"][1]["iters"]
+    rel = np.linalg.norm(res["ref"][0] - res["p2p"][0]) / np.linalg.norm(res["ref"][0])
+    assert rel < 1e-12
 
 
 def test_p2p_loopback_solve(torch_cuda):

@@ -69,6 +69,19 @@ def test_partitioned_bitwise_p2p_halo(torch_cuda, tmp_path, n):
     assert res["ok"], (bad, res.get("solve"))
 
 
+@pytest.mark.parametrize("n,grid", [(2, "1,1,2,1"), (4, "1,1,2,2"), (4, "2,1,1,2")])
+def test_grid_partitioned_bitwise_p2p_halo(torch_cuda, tmp_path, n, grid):
+    """Kernel-initiated halo of a process grid between processes (CUDA IPC mappings on one GPU;
+    NVLink peers on a multi-GPU node): one pack kernel per operator stores every split
+    dimension's faces into the neighbours' ghosts and raises their flags; the solver's sums go
+    through the kernel-side allreduce.  Bitwise = unpartitioned; solve meets the oracle."""
+    r, out = _run(n, "host", tmp_path, "8,4,8,16", halo="p2p", grid=grid)
+    assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
+    res = json.load(open(out))
+    bad = [k for k, v in res["checks"].items() if not v]
+    assert res["ok"], (bad, res.get("solve"))
+
+
 def test_partitioned_nccl_distinct_gpus(torch_cuda, tmp_path):
     import torch
     if torch.cuda.device_count() < 2:

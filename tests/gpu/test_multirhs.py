@@ -61,3 +61,67 @@ def test_multirhs_fused_reductions_match_single(torch_cuda):
     with pytest.raises(qudax.QudaxError):
         ctx.solve_multi([qgen.point_source(dims, 0, 0)], use_schur=2)
     ctx.close()
+
+
+@pytest.mark.parametrize("prec,recon", [(4, 12), (2, 12), (8, 18)])
+@pytest.mark.parametrize("overlap", [True, False])
+def test_multi_rhs_halo_loopback_bitwise(torch_cuda, prec, recon, overlap):
+    """The multi-RHS T halo (one exchange per direction carries every right-hand side's face;
+    interior / boundary ranges of the multi-RHS kernel) through NCCL loopback at N = 1: every
+    kind and dagger bitwise equal to the unpartitioned multi-RHS launch (the exchange moves bits
+    only and the per-site code is the same)."""
+    dims = (8, 4, 6, 8)
+    nrhs = 3
+    U = qgen.gauge(dims, 1411)
+    psis = [qgen.spinor(dims, 1600 + k) for k in range(nrhs)]
+    outs = {}
+    for comm in (qudax.COMM_NONE, qudax.COMM_NCCL):
+        ctx = qudax.Context(dims, comm=comm, overlap=overlap, nccl_id=qudax.nccl_unique_id() if comm else None)
+        ctx.gauge_load(U, 0.12, 1.0, prec=prec, recon=recon)
+        ins = [ctx.new_field(prec) for _ in range(nrhs)]
+        xs = [ctx.new_field(prec) for _ in range(nrhs)]
+        for k in range(nrhs):
+            ctx.spinor_load(ins[k], prec, 1, psis[k])
+            ctx.spinor_load(xs[k], prec, 0, psis[(k + 1) % nrhs])
+        res = []
+        for dagger in (False, True):
+            for kind in (0, 1, 2, 3):
+                o = [ctx.new_field(prec) for _ in range(nrhs)]
+                ctx.dslash_multi(o, ins, prec, 0, dagger=dagger, kind=kind, xs=xs, a=-0.3)
+                ctx.sync()
+                res += [f.cpu().numpy().copy() for f in o]
+        ev = [ctx.new_field(prec) for _ in range(nrhs)]
+        for k in range(nrhs):
+            ctx.spinor_load(ev[k], prec, 0, psis[k])
+        o = [ctx.new_field(prec) for _ in range(nrhs)]
+        ctx.matpc_multi(o, ev, prec)
+        ctx.sync()
+        res += [f.cpu().numpy().copy() for f in o]
+        outs[comm] = res
+        ctx.close()
+    for a, b in zip(outs[qudax.COMM_NONE], outs[qudax.COMM_NCCL]):
+        assert np.array_equal(a, b)
+
+
+def test_batched_solve_loopback_multi_rhs_halo(torch_cuda):
+    """Batched solve through the multi-RHS halo + per-RHS ncclAllReduce (NCCL loopback, no
+    overlap so the reductions keep the unsplit CTA grouping): bitwise the unpartitioned batched
+    solve, and each system bitwise its own single solve."""
+    dims = (8, 8, 8, 16)
+    U = qgen.gauge(dims, 1003, eps=0.1)
+    srcs = [qgen.point_source(dims, s, c) for s, c in ((0, 0), (1, 2), (0, 1))]
+    res = {}
+    for comm in (qudax.COMM_NONE, qudax.COMM_NCCL):
+        ctx = qudax.Context(dims, comm=comm, overlap=False, nccl_id=qudax.nccl_unique_id() if comm else None)
+        ctx.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+        xs, sts = ctx.solve_multi(srcs, tol=1e-10, delta=1e-2, maxiter=2000, prec=8, prec_sloppy=4)
+        res[comm] = (xs, [s["iters"] for s in sts])
+        if comm == qudax.COMM_NCCL:
+            for j, b in enumerate(srcs):
+                x1, st1 = ctx.solve(b, tol=1e-10, delta=1e-2, maxiter=2000, prec=8, prec_sloppy=4)
+                assert st1["iters"] == sts[j]["iters"]
+                assert np.array_equal(x1, xs[j])
+        ctx.close()
+    assert res[qudax.COMM_NONE][1] == res[qudax.COMM_NCCL][1]
+    for a, b in zip(res[qudax.COMM_NONE][0], res[qudax.COMM_NCCL][0]):
+        assert np.array_equal(a, b)
