@@ -459,20 +459,6 @@ __host__ __device__ constexpr bool dslash_pair() {
     return P == 8 || (P == 2 && RECON != 12);
 #endif
 }
-// Whether the unpartitioned kernel runs its 8 hops as a software pipeline: the raw operands of
-// hop k+1 (neighbour spinor + link, still packed) are loaded before hop k is decoded and
-// computed, so one hop's loads are always in flight (dslash_pair only overlaps the two hops of
-// one direction, then waits).  The half kernel was memory-latency bound at its register-capped
-// occupancy (ncu r01k: stall samples on the first PRMT after every hop's loads).
-// QX_PIPE_MASK overrides: bit 0 half, 1 fp32, 2 fp64.
-template <int P, int RECON>
-__host__ __device__ constexpr bool dslash_pipe() {
-#ifdef QX_PIPE_MASK
-    return (QX_PIPE_MASK >> (P == 2 ? 0 : (P == 4 ? 1 : 2))) & 1;
-#else
-    return P == 2;
-#endif
-}
 #ifndef QX_DSLASH_THREADS
 #define QX_DSLASH_THREADS 128
 #endif
@@ -505,24 +491,6 @@ __device__ __forceinline__ void pf_spinor_l1(const void *base, long stride, long
         for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + j)));
     }
 }
-// L1 prefetch of a site's clover (CLOVER_INV reads it only after the 8 hops): issued before the
-// temporal hops, the epilogue's streamed loads then hit L1 instead of paying a DRAM round trip
-// after the last hop.  QX_CLV_PF: 1 on (default for the pipelined half kernel), 0 off.
-#ifndef QX_CLV_PF
-#define QX_CLV_PF 1
-#endif
-template <int P>
-__device__ __forceinline__ void pf_clover_l1(const void *base, long stride, long i) {
-    if constexpr (P == 2) {
-#pragma unroll
-        for (int k = 0; k < 9; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + i)));
-        pf_l1(cptr(base, (size_t)144 * stride + 8 * i));
-    } else {
-        constexpr int NB = (P == 8) ? 36 : 18;
-#pragma unroll
-        for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + i)));
-    }
-}
 // one output site; red[] receives this site's contribution to the optional fused reduction
 // INMODE: load mode of the neighbour spinors (0 read-only path; 2 L2-coherent, for inputs
 // written by other CTAs earlier in the same launch — the fused Mhat kernel)
@@ -530,7 +498,7 @@ __device__ __forceinline__ void pf_clover_l1(const void *base, long stride, long
 // separate instantiation so the unpartitioned kernels keep their register allocation
 template <int P, int RECON, bool DAG, int KIND, int INMODE = 0, bool SS = false>
 __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin, void *fout, const void *fx, int tid,
-                                            double red[3], long goff = 0, int sbit = 0) {
+                                            double red[3], long goff = 0, int sbit = 0, int hv = 0) {
     using R = typename Prec<P>::R;
     if (a.reverse) tid = a.nthreads - 1 - tid;
     const int X = a.X, Y = a.Y, Z = a.Z, Xh = a.Xh;
@@ -601,6 +569,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // flight per thread (dslash_pair).
     constexpr bool PAIR = dslash_pair<P, RECON>();
     constexpr bool DF = dslash_defer<P, RECON>();
+    bool bail = false;
     auto spatial = [&](auto mu_c, int coord, int Lmu, int nf, int nb) {
         constexpr int MU = decltype(mu_c)::value;
         // operand sources of the two hops: the input field, or (partitioned X) the neighbour's
@@ -673,6 +642,15 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             sb.template load_spinor<INMODE>(bsrc, bstr, nb);
             lb.load(lbsrc, lbstr, lbi);
         }
+        if constexpr (MU == 0) {
+            // a halted solver batch (SolverScalars::halt): the flag was loaded at kernel entry and
+            // is tested only here, after the first hop's loads are in flight, so its latency is
+            // not added to every thread's critical path
+            if (hv) {
+                bail = true;
+                return;
+            }
+        }
         if constexpr (DF && QX_BPROJ) {
             R v[24];
             Cx<R> ps[4][3], u[3][3], h0[3], h1[3];
@@ -714,104 +692,8 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     const int nxf = (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1, nxb = (x == 0 ? lex + (X - 1) : lex - 1) >> 1;
     const int nyf = (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1, nyb = (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1;
     const int nzf = (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1, nzb = (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1;
-    constexpr bool PIPE = !SS && dslash_pipe<P, RECON>();
-    if constexpr (PIPE) {
-        // ---- software-pipelined hops (dslash_pipe): load hop k+1, then compute hop k
-        const int T_loc = a.T_loc;
-        constexpr bool FWD_UPPER = (SF > 0), BWD_UPPER = (SB > 0);
-        const bool fwd_ghost = (t == T_loc - 1) && a.ghosted;
-        const bool bwd_ghost = (t == 0) && a.ghosted;
-        const R cft = (t == T_loc - 1) ? (R)(2.0 * a.bc_fwd) : (R)2;
-        const R cbt = (t == 0) ? (R)(2.0 * a.bc_back) : (R)2;
-        const int nfw = (t == T_loc - 1 ? lex - (T_loc - 1) * XYZ : lex + XYZ) >> 1;
-        const int nbw = (t == 0 ? lex + (T_loc - 1) * XYZ : lex - XYZ) >> 1;
-        struct SpHop {
-            RawVec<P, 24> s;
-            RawLink<P, RECON> l;
-        };
-        struct THop {
-            RawVec<P, 12> s;
-            RawLink<P, RECON> l;
-        };
-        auto load_sp = [&](SpHop &h, int mu, bool fwd, int n) {
-            h.s.template load_spinor<INMODE>(fin, a.stride, n);
-            if (fwd) h.l.load(a.gauge[mu][p], a.stride, i);
-            else h.l.load(a.gauge[mu][op], a.stride, n);
-        };
-        auto comp_sp = [&](const SpHop &h, auto mu_c, auto sg_c) {
-            constexpr int MU = decltype(mu_c)::value, SG = decltype(sg_c)::value;
-            constexpr bool ADJ = (SG == SB);  // the backward hop applies U(x - mu)^dag
-            R v[24];
-            Cx<R> ps[4][3], u[3][3];
-            if constexpr (DF && QX_BPROJ) {
-                Cx<R> h0[3], h1[3];
-                h.s.decode_b(v);
-                unpack_spinor(v, ps);
-                spatial_project_b<MU, SG>(ps, h0, h1);
-                const R sc = h.s.scale() * dec_link<DF>(h.l, u);
-                spatial_mult_expand<MU, SG, ADJ, DF>(h0, h1, u, acc, sc);
-            } else {
-                R sc = dec_vec<DF>(h.s, v);
-                unpack_spinor(v, ps);
-                sc *= dec_link<DF>(h.l, u);
-                spatial_hop<MU, SG, ADJ, DF>(ps, u, acc, sc);
-            }
-        };
-        auto load_tf = [&](THop &h) {
-            if (fwd_ghost) h.s.load_face(static_cast<const char *>(a.ghost_fwd) + goff, a.fstride, i - t * a.F);
-            else h.s.template load_half<INMODE>(fin, a.stride, nfw, FWD_UPPER ? 0 : 1);
-            h.l.load(a.gauge[3][p], a.stride, i);
-        };
-        auto load_tb = [&](THop &h) {
-            if (bwd_ghost) {
-                h.s.load_face(static_cast<const char *>(a.ghost_back) + goff, a.fstride, i);
-                h.l.load(a.gauge_ghost, a.fstride, i);
-            } else {
-                h.s.template load_half<INMODE>(fin, a.stride, nbw, BWD_UPPER ? 0 : 1);
-                h.l.load(a.gauge[3][op], a.stride, nbw);
-            }
-        };
-        auto comp_t = [&](const THop &h, auto up_c, auto adj_c, R coef) {
-            R hv[12];
-            Cx<R> u[3][3];
-            R sc = dec_vec<DF>(h.s, hv);
-            sc *= dec_link<DF>(h.l, u);
-            temporal_hop<decltype(up_c)::value, decltype(adj_c)::value>(hv, u, DF ? coef * sc : coef, acc);
-        };
-        using I0 = std::integral_constant<int, 0>;
-        using I1 = std::integral_constant<int, 1>;
-        using I2 = std::integral_constant<int, 2>;
-        using CF = std::integral_constant<int, SF>;
-        using CB = std::integral_constant<int, SB>;
-        SpHop A, B;
-        load_sp(A, 0, true, nxf);
-        load_sp(B, 0, false, nxb);
-        comp_sp(A, I0{}, CF{});
-        load_sp(A, 1, true, nyf);
-        comp_sp(B, I0{}, CB{});
-        load_sp(B, 1, false, nyb);
-        comp_sp(A, I1{}, CF{});
-        load_sp(A, 2, true, nzf);
-        comp_sp(B, I1{}, CB{});
-        load_sp(B, 2, false, nzb);
-        comp_sp(A, I2{}, CF{});
-        THop C, D;
-        load_tf(C);
-#if QX_CLV_PF
-        if constexpr (KIND == QUDAX_CLOVER_INV || KIND == QUDAX_CLOVER_INV_XPAY) pf_clover_l1<P>(a.clover, a.stride, i);
-#endif
-        comp_sp(B, I2{}, CB{});
-        load_tb(D);
-#if QX_RED_PF
-        if (a.red_kind != RED_NONE) {
-            const void *w = a.red_kind == RED_XDOT_NORM ? fx : (a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat);
-            pf_spinor_l1<P>(w, a.stride, i);
-        }
-#endif
-        comp_t(C, std::bool_constant<FWD_UPPER>{}, std::false_type{}, cft);
-        comp_t(D, std::bool_constant<BWD_UPPER>{}, std::true_type{}, cbt);
-    } else {
     spatial(std::integral_constant<int, 0>{}, x, X, nxf, nxb);
+    if (bail) return;
     spatial(std::integral_constant<int, 1>{}, y, Y, nyf, nyb);
     spatial(std::integral_constant<int, 2>{}, z, Z, nzf, nzb);
 
@@ -872,7 +754,6 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             temporal_hop<BWD_UPPER, true>(h, u, DF ? cb * sc : cb, acc);
         }
     }
-    }  // !PIPE
 
     // ---- epilogue: fused clover
     Cx<R> res[4][3];
@@ -985,7 +866,17 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     // hardware CTA scheduler balances the memory-latency-bound CTAs better than a fixed wave)
     // multi-RHS (a.nrhs > 1): consecutive CTAs take the same sites for different right-hand
     // sides, so the links and clover they stream are served from L2 after the first of them
-    if (halted(a.halt)) return;  // the rest of a solver batch after a reliable-update request
+#ifndef QX_HALT_LATE
+#define QX_HALT_LATE 1
+#endif
+#if QX_HALT_LATE
+    // the rest of a solver batch after a reliable-update request does nothing: the flag is read
+    // now and tested after the first hop's loads are issued (dslash_site)
+    const int hv = a.halt ? *reinterpret_cast<const volatile int *>(a.halt) : 0;
+#else
+    if (halted(a.halt)) return;
+    const int hv = 0;
+#endif
     int blk = blockIdx.x, rhs = 0;
     if (a.nrhs > 1) {
         rhs = blk % a.nrhs;
@@ -1000,10 +891,12 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kerne
     int sbit = 0;                               // kernel-initiated halo: sequence parity of the ghosts
     // RANGE_TAIL: only CTAs holding boundary sites (the grid's last ones) wait for the halo
     if (a.p2p_flags && (a.range != RANGE_TAIL || (blk + 1) * (int)blockDim.x > a.tail_ni)) {
+        if (hv) return;  // (the matching pack kernel was halted too: no flag to wait for)
         sbit = p2p_wait(a);
         goff = sbit ? a.p2p_pdist : 0L;
     }
-    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND, 0, SS>(a, fin, fout, fx, tid, red, goff, sbit);
+    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND, 0, SS>(a, fin, fout, fx, tid, red, goff, sbit, hv);
+    if (hv) return;
     if (a.p2p_flags) {  // the last CTA to finish advances the consumed-halo counter
         __syncthreads();
         if (threadIdx.x == 0 && atomicAdd(a.p2p_ccount, 1u) == gridDim.x - 1) {

@@ -103,16 +103,22 @@ static cudaGraphExec_t capture_graph(qudax_ctx *c, F &&body, long long *nlaunch,
         if (g) cudaGraphDestroy(g);
         c->capturing = false;
         c->cap_iter = 0;
+        c->launches = l0;
         release_graph_timing(c, c->graph_trecs);
         throw;
     }
-    cudaGraph_t graph;
-    QX_CUDA(cudaStreamEndCapture(c->stream, &graph));
+    cudaGraph_t graph = nullptr;
+    const cudaError_t ee = cudaStreamEndCapture(c->stream, &graph);
     c->capturing = false;
     c->cap_iter = 0;
-    cudaGraphExec_t exec;
-    QX_CUDA(cudaGraphInstantiate(&exec, graph, 0));
-    cudaGraphDestroy(graph);
+    cudaGraphExec_t exec = nullptr;
+    const cudaError_t ie = (ee == cudaSuccess) ? cudaGraphInstantiate(&exec, graph, 0) : ee;
+    if (graph) cudaGraphDestroy(graph);
+    if (ie != cudaSuccess) {
+        c->launches = l0;
+        release_graph_timing(c, c->graph_trecs);
+        throw Error(QUDAX_ERR_CUDA, std::string("solver graph capture: ") + cudaGetErrorString(ie));
+    }
     *nlaunch = c->launches - l0;
     c->launches = l0;
     trecs->swap(c->graph_trecs);
@@ -131,11 +137,11 @@ void drop_graphs(qudax_ctx *c) {
     c->graphs.clear();
 }
 template <typename F>
-static qudax_ctx::Graph &cached_graph(qudax_ctx *c, std::vector<uintptr_t> key, F &&body) {
+static qudax_ctx::Graph *cached_graph(qudax_ctx *c, std::vector<uintptr_t> key, F &&body) {
     key.push_back((uintptr_t)c->gauge_epoch);
     key.push_back((uintptr_t)c->timing);
     for (auto &gr : c->graphs)
-        if (gr.key == key) return gr;
+        if (gr.key == key) return &gr;
     if (c->graphs.size() >= kMaxGraphs) {
         auto &old = c->graphs.front();
         if (old.exec) cudaGraphExecDestroy(old.exec);
@@ -144,9 +150,19 @@ static qudax_ctx::Graph &cached_graph(qudax_ctx *c, std::vector<uintptr_t> key, 
     }
     qudax_ctx::Graph gr;
     gr.key = std::move(key);
-    gr.exec = capture_graph(c, body, &gr.launches, &gr.trecs);
+    try {
+        gr.exec = capture_graph(c, body, &gr.launches, &gr.trecs);
+    } catch (const Error &e) {
+        // a capture the runtime or a transport refuses (e.g. a NCCL build without graph support):
+        // the context continues with eager enqueues, which compute the same iterates
+        if (e.status != QUDAX_ERR_CUDA && e.status != QUDAX_ERR_NCCL) throw;
+        cudaGetLastError();
+        std::fprintf(stderr, "qudax: CUDA-graph capture of the solver batch failed (%s); continuing eagerly\n", e.what());
+        c->flags |= QUDAX_FLAG_NO_GRAPHS;
+        return nullptr;
+    }
     c->graphs.push_back(std::move(gr));
-    return c->graphs.back();
+    return &c->graphs.back();
 }
 
 // RAII: kernels launched while this is alive carry the solver batch gate
@@ -339,10 +355,14 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
             const std::vector<uintptr_t> key = {1, (uintptr_t)Pd, (uintptr_t)Ps, (uintptr_t)batch, (uintptr_t)rs,
                                                 (uintptr_t)xs, (uintptr_t)p, (uintptr_t)v, (uintptr_t)t,
                                                 (uintptr_t)r0, (uintptr_t)S, (uintptr_t)c->matpc_sym};
-            auto &gr = cached_graph(c, key, [&] { enqueue_batch(batch); });
-            QX_CUDA(cudaGraphLaunch(gr.exec, c->stream));
-            c->launches += gr.launches;
-            grecs = &gr.trecs;
+            auto *gr = cached_graph(c, key, [&] { enqueue_batch(batch); });
+            if (gr) {
+                QX_CUDA(cudaGraphLaunch(gr->exec, c->stream));
+                c->launches += gr->launches;
+                grecs = &gr->trecs;
+            } else {
+                enqueue_batch(batch);
+            }
         }
         QX_CUDA(cudaMemcpyAsync(hS, S, sizeof(*hS), cudaMemcpyDeviceToHost, c->stream));
         QX_CUDA(cudaStreamSynchronize(c->stream));
@@ -538,10 +558,14 @@ void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_
                                           (uintptr_t)c->d_scal_m};
             for (int j = 0; j < n; ++j)
                 for (void *f : {sys[j].rs, sys[j].xs, sys[j].p, sys[j].v, sys[j].t, sys[j].r0}) key.push_back((uintptr_t)f);
-            auto &gr = cached_graph(c, key, [&] { enqueue_iteration(mask); });
-            QX_CUDA(cudaGraphLaunch(gr.exec, c->stream));
-            c->launches += gr.launches;
-            grecs = &gr.trecs;
+            auto *gr = cached_graph(c, key, [&] { enqueue_iteration(mask); });
+            if (gr) {
+                QX_CUDA(cudaGraphLaunch(gr->exec, c->stream));
+                c->launches += gr->launches;
+                grecs = &gr->trecs;
+            } else {
+                enqueue_iteration(mask);
+            }
         }
         QX_CUDA(cudaStreamSynchronize(c->stream));
         if (grecs) harvest_graph_timing(c, *grecs, 1);
