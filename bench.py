@@ -45,7 +45,7 @@ BLAS_FLOPS_PER_SITE_ITER = 960.0
 def parse():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
-    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--steps", type=int, default=20)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--iters", type=int, default=100, help="BiCGstab iterations per step")
@@ -56,6 +56,10 @@ def parse():
                     help="N>1 spinor halo: NCCL send/recv (comm) or kernel-initiated over peer memory (p2p)")
     ap.add_argument("--grid", default="", help="process grid Px,Py,Pz,Pt (default 1,1,1,N: T slabs, P:563-605; "
                                                "others: multi-dimensional split, SURVEY 8(f) item 4)")
+    ap.add_argument("--no-kernel-timing", action="store_true",
+                    help="diagnostic: no per-launch CUDA events in the timed region (no roofline)")
+    ap.add_argument("--breakdown", action="store_true",
+                    help="diagnostic: per (precision, kind, fused reduction) in-step Dslash times to stderr")
     ap.add_argument("--scaling", default="weak", choices=["weak", "strong"],
                     help="weak: 32^3x64 per GPU (BASELINE configs[4]); strong: 32^3x256 in total (configs[3])")
     ap.add_argument("--oracle-sample", type=int, default=0, help=argparse.SUPPRESS)  # internal: 1-thread oracle run
@@ -424,7 +428,7 @@ def main():
                             overlap=bool(args.overlap), proc_grid=grid,
                             halo=qudax.HALO_P2P if args.halo == "p2p" else qudax.HALO_COMM)
     else:
-        ctx = qudax.Context(dims, device=local)
+        ctx = qudax.Context(dims, device=local, flags=qudax.FLAG_TIMING_BREAKDOWN if args.breakdown else 0)
     assert ctx.local_dims == local_dims, (ctx.local_dims, local_dims)
     origin = ctx.partition["origin"]
     U = qgen.gauge_box(dims, GAUGE_SEED, origin, local_dims, eps=EPS)
@@ -446,7 +450,7 @@ def main():
 
     # ---- timed region (device-resident inputs)
     l0 = ctx.launch_count()
-    ctx.kernel_timing(True)
+    ctx.kernel_timing(not args.no_kernel_timing)
     flops = 0.0
     iters = 0
     updates = 0

@@ -552,7 +552,8 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
             c->launches += 1;
         };
         const bool sp = spatial_split(g) != 0;
-        const bool tail = c->overlap && (sp || g.T_loc > 2);
+        // (a split X has no interior box: every site may read a ghost, so every CTA waits)
+        const bool tail = c->overlap && (sp ? g.n_int > 0 : g.T_loc > 2);
         if (tail) {
             // ONE Dslash launch (RANGE_TAIL) beside the pack on the high-priority comm stream:
             // interior sites first (T-only: t in [1, T_loc-2]; a grid: the interior box), the
