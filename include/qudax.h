@@ -277,6 +277,14 @@ qudax_status qudax_get_partition(const qudax_ctx *ctx, qudax_partition *out);
 qudax_status qudax_kernel_timing(qudax_ctx *ctx, int enable);
 /* Synchronise and sum the recorded Dslash launches of precision prec_filter (0 = all). */
 qudax_status qudax_get_kernel_stats(qudax_ctx *ctx, int prec_filter, qudax_kernel_stats *out);
+/* Diagnostic timeline of the halo overlap on the NCCL path.  enable = 1: every
+ * subsequent eagerly launched split Dslash records CUDA events on both streams; out7 (may be
+ * NULL) receives, for the last recorded call, the microseconds from its start (compute stream)
+ * to: pack start, exchange start, exchange end (comm stream), interior kernel start, interior
+ * end, boundary kernel start, boundary end (compute stream).  Without an interior/boundary split
+ * (overlap off) the three "interior" marks coincide with the boundary start.  enable = 0 stops
+ * recording.  QUDAX_ERR_STATE if nothing was recorded. */
+qudax_status qudax_halo_timeline(qudax_ctx *ctx, int enable, double *out7);
 
 /* ---- gauge field and clover (setup) ----
  * Uploads the host box, exchanges a one-site gauge halo (with corners: one dimension after the

@@ -606,20 +606,38 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         }
     };
     if (c->comm == QUDAX_COMM_NCCL) {
+        // diagnostic overlap timeline (qudax_halo_timeline), eager launches only
+        const bool tl = c->tl_on && !c->capturing;
+        auto mark = [&](int k, cudaStream_t st) {
+            if (tl) QX_CUDA(cudaEventRecord(c->tl[k], st));
+        };
         // comm stream: wait for `in` (and for the previous boundary kernel, which read the ghosts)
+        mark(0, c->stream);
         QX_CUDA(cudaEventRecord(c->ev_in, c->stream));
         QX_CUDA(cudaStreamWaitEvent(c->comm_stream, c->ev_in, 0));
+        mark(1, c->comm_stream);
         pack_all(c->comm_stream);
+        mark(2, c->comm_stream);
         exchange_all(c, xf, nx, c->comm_stream);
+        mark(3, c->comm_stream);
         QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
         if (split) {
+            mark(4, c->stream);
             launch(RANGE_INTERIOR, (int)n_int);
+            mark(5, c->stream);
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
+            mark(6, c->stream);
             launch(RANGE_BOUNDARY, (int)n_bnd);
+            mark(7, c->stream);
         } else {
             QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
+            mark(4, c->stream);
+            mark(5, c->stream);
+            mark(6, c->stream);
             launch(RANGE_ALL, (int)g.Vh);
+            mark(7, c->stream);
         }
+        if (tl) c->tl_valid = true;
     } else {  // HOST: paper strategy 1 (no overlap)
         pack_all(c->stream);
         exchange_all(c, xf, nx, c->stream);
@@ -1452,6 +1470,8 @@ qudax_status qudax_finalize(qudax_ctx *c) {
     for (auto e : c->ev_pool) cudaEventDestroy(e);
     for (auto e : c->xfer.done)
         if (e) cudaEventDestroy(e);
+    for (auto e : c->tl)
+        if (e) cudaEventDestroy(e);
     if (c->ev_in) cudaEventDestroy(c->ev_in);
     if (c->ev_halo) cudaEventDestroy(c->ev_halo);
     if (c->comm_stream) cudaStreamDestroy(c->comm_stream);
@@ -1521,6 +1541,25 @@ qudax_status qudax_get_kernel_stats(qudax_ctx *c, int prec_filter, qudax_kernel_
             o->bytes_compulsory += t.bytes_c;
             o->bytes_paper += t.bytes_p;
         }
+    });
+}
+
+qudax_status qudax_halo_timeline(qudax_ctx *c, int enable, double *out7) {
+    if (!c) return QUDAX_ERR_ARG;
+    return guard(c, [&] {
+        if (out7) {
+            QX_CHECK(c->tl_valid, QUDAX_ERR_STATE, "halo timeline: no split Dslash recorded");
+            QX_CUDA(cudaStreamSynchronize(c->stream));
+            QX_CUDA(cudaStreamSynchronize(c->comm_stream));
+            for (int k = 1; k < 8; ++k) {
+                float ms = 0;
+                QX_CUDA(cudaEventElapsedTime(&ms, c->tl[0], c->tl[k]));
+                out7[k - 1] = 1e3 * ms;
+            }
+        }
+        if (enable && !c->tl[0])
+            for (auto &e : c->tl) QX_CUDA(cudaEventCreate(&e));
+        c->tl_on = enable != 0;
     });
 }
 

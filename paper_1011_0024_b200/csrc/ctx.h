@@ -15,6 +15,9 @@ struct qudax_ctx {
     cudaStream_t stream = nullptr, comm_stream = nullptr;
     bool own_stream = false;
     cudaEvent_t ev_in = nullptr, ev_halo = nullptr;
+    // diagnostic halo-overlap timeline (qudax_halo_timeline)
+    bool tl_on = false, tl_valid = false;
+    cudaEvent_t tl[8] = {};
     ncclComm_t nccl = nullptr;
     qudax_alloc_fn dev_alloc = nullptr;
     qudax_free_fn dev_free = nullptr;

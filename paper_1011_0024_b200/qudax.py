@@ -126,6 +126,7 @@ SIGNATURES = {
     "qudax_get_partition": ([_P, ctypes.POINTER(Partition)], _I),
     "qudax_kernel_timing": ([_P, _I], _I),
     "qudax_get_kernel_stats": ([_P, _I, ctypes.POINTER(KernelStats)], _I),
+    "qudax_halo_timeline": ([_P, _I, _DP], _I),
     "qudax_gauge_load": ([_P, _DP, ctypes.POINTER(GaugeParam)], _I),
     "qudax_spinor_bytes": ([_P, _I], _Z),
     "qudax_spinor_load": ([_P, _P, _I, _I, _DP], _I),
@@ -385,6 +386,18 @@ class Context:
 
     def kernel_timing(self, enable=True):
         self._check(lib().qudax_kernel_timing(self._h, int(bool(enable))))
+
+    def halo_timeline(self, enable=True, read=False):
+        """Diagnostic halo-overlap timeline (NCCL path): enable recording; with read=True return
+        the last recorded call's marks (µs from its start): pack start, exchange start, exchange
+        end, interior start, interior end, boundary start, boundary end."""
+        out = (ctypes.c_double * 7)() if read else None
+        self._check(lib().qudax_halo_timeline(self._h, int(bool(enable)), out))
+        if read:
+            keys = ("pack_start", "exchange_start", "exchange_end", "interior_start", "interior_end",
+                    "boundary_start", "boundary_end")
+            return dict(zip(keys, list(out)))
+        return None
 
     def kernel_stats(self, prec=0):
         out = KernelStats()

@@ -190,3 +190,25 @@ def test_loopback_split_dims_solve(torch_cuda):
         c.close()
     assert res["ref"][1]["iters"] == res["split"][1]["iters"]
     assert np.array_equal(res["ref"][0], res["split"][0])
+
+
+def test_halo_timeline_shows_overlap(torch_cuda):
+    """The NCCL path's pack + exchange run on the comm stream while the interior kernel runs on
+    the compute stream: events on both streams (qudax_halo_timeline) must show the
+    comm-stream work starting before the interior kernel ends, and the boundary kernel starting
+    only after the exchange ended."""
+    dims = (16, 16, 16, 32)
+    ctx = qudax.Context(dims, comm=qudax.COMM_NCCL, nccl_id=qudax.nccl_unique_id(), overlap=True)
+    ctx.gauge_load(qgen.gauge(dims, 1261), 0.12, 1.0, prec=4, recon=12)
+    fi, fo = ctx.new_field(4), ctx.new_field(4)
+    ctx.spinor_load(fi, 4, 0, qgen.spinor(dims, 1262))
+    ctx.matpc(fo, fi, 4)
+    ctx.halo_timeline(True)
+    ctx.matpc(fo, fi, 4)
+    m = ctx.halo_timeline(False, read=True)
+    ctx.close()
+    order = ["pack_start", "exchange_start", "exchange_end"]
+    assert all(m[a] <= m[b] for a, b in zip(order, order[1:])), m
+    assert m["interior_start"] <= m["interior_end"] <= m["boundary_start"] <= m["boundary_end"], m
+    assert m["pack_start"] < m["interior_end"], m        # the halo work began while the interior ran
+    assert m["boundary_start"] >= m["exchange_end"], m   # the boundary waited for the ghosts
