@@ -845,7 +845,7 @@ static void global_sum(qudax_ctx *c, double *dev_vals, int n, double *res) {
         return;
     }
     if (c->comm == QUDAX_COMM_NCCL) {  // (one rank: the loopback test of the N > 1 path)
-        QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl, c->stream));
+        QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl_red, c->stream));
     }
     QX_CUDA(cudaMemcpyAsync(c->h_red, dev_vals, sizeof(double) * n, cudaMemcpyDeviceToHost, c->stream));
     QX_CUDA(cudaStreamSynchronize(c->stream));
@@ -872,7 +872,7 @@ int blas_op(qudax_ctx *c, int op, int prec, void *const *f, const double *coef, 
 // rank), then the device-side scalar recurrence `mode` (launch_coef).
 void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, int mode) {
     if (c->comm == QUDAX_COMM_NCCL) {  // (one rank: the loopback test of the N > 1 path)
-        QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl, c->stream));
+        QX_NCCL(ncclAllReduce(dev_vals, dev_vals, n, ncclDouble, ncclSum, c->nccl_red, c->stream));
     } else if (c->g.nranks > 1 && c->comm == QUDAX_COMM_HOST) {
         QX_CUDA(cudaMemcpyAsync(c->h_red, dev_vals, sizeof(double) * n, cudaMemcpyDeviceToHost, c->stream));
         QX_CUDA(cudaStreamSynchronize(c->stream));
@@ -1199,7 +1199,7 @@ static void allgather_small(qudax_ctx *c, const void *mine, size_t n, void *all)
     if (c->comm == QUDAX_COMM_NCCL) {
         char *d = static_cast<char *>(dalloc(c, n * (g.nranks + 1)));
         QX_CUDA(cudaMemcpyAsync(d, mine, n, cudaMemcpyHostToDevice, c->stream));
-        QX_NCCL(ncclAllGather(d, d + n, n, ncclChar, c->nccl, c->stream));
+        QX_NCCL(ncclAllGather(d, d + n, n, ncclChar, c->nccl_red, c->stream));
         QX_CUDA(cudaMemcpyAsync(all, d + n, n * g.nranks, cudaMemcpyDeviceToHost, c->stream));
         QX_CUDA(cudaStreamSynchronize(c->stream));
         dfree(c, d);
@@ -1395,6 +1395,12 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
             ncclUniqueId id;
             std::memcpy(&id, p->nccl_id, sizeof(id));
             QX_NCCL(ncclCommInitRank(&c->nccl, g.nranks, id, g.rank));
+            // a second communicator for the global sums: the halo's send/recv run on the comm
+            // stream and the allreduces on the compute stream, and operations of ONE communicator
+            // issued from two streams may be serialised by NCCL in an order that deadlocks against
+            // the streams' own event dependencies (seen: the loopback solve with a Y/Z/T split
+            // hung once its sums went through NCCL)
+            QX_NCCL(ncclCommSplit(c->nccl, 0, g.rank, &c->nccl_red, nullptr));
         }
         c->partials = static_cast<double *>(dalloc(c, sizeof(double) * 4 * blas_partial_blocks()));
         c->red_out = static_cast<double *>(dalloc(c, sizeof(double) * 8));
@@ -1458,6 +1464,7 @@ qudax_status qudax_finalize(qudax_ctx *c) {
     for (char *m : c->p2p.opened)
         if (m) cudaIpcCloseMemHandle(m);
     if (c->p2p.base) cudaFree(c->p2p.base);
+    if (c->nccl_red) ncclCommDestroy(c->nccl_red);
     if (c->nccl) ncclCommDestroy(c->nccl);
     for (void *p : c->allocs) {
         if (c->dev_free) c->dev_free(p, c->alloc_user);

@@ -18,7 +18,8 @@ struct qudax_ctx {
     // diagnostic halo-overlap timeline (qudax_halo_timeline)
     bool tl_on = false, tl_valid = false;
     cudaEvent_t tl[8] = {};
-    ncclComm_t nccl = nullptr;
+    ncclComm_t nccl = nullptr;      // halo send/recv (comm stream) and setup exchanges
+    ncclComm_t nccl_red = nullptr;  // global sums (compute stream): split from nccl
     qudax_alloc_fn dev_alloc = nullptr;
     qudax_free_fn dev_free = nullptr;
     void *alloc_user = nullptr;
