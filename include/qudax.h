@@ -248,6 +248,9 @@ typedef struct {
     double flops;                /* effective flops of those launches (qudax_model per kind) */
     double bytes_compulsory;     /* algorithmic bytes (compulsory model) of those launches */
     double bytes_paper;          /* paper-model bytes */
+    double span_ms_total;        /* sum of the launches' in-kernel spans: %globaltimer of the first CTA
+                                    to start to that of the last CTA to finish (the kernel's own
+                                    execution time, without the launch bubble of the events) */
 } qudax_kernel_stats;
 
 /* ---- host-only helpers (no GPU needed) ---- */

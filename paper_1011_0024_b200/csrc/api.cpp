@@ -343,13 +343,23 @@ static void launch_dslash_raw(int prec, int recon, int dagger, int kind, const D
 
 // every Dslash kernel launch goes through here; with timing enabled it is bracketed by CUDA
 // events on the launching (compute) stream
-static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int kind, const DslashArgs &a) {
+constexpr int kSpanSlots = 1 << 14;
+static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int kind, const DslashArgs &a0) {
     if (!c->timing) {
-        launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
+        launch_dslash_raw(prec, recon, dagger, kind, a0, c->stream);
         return;
     }
+    if (!c->d_span) {
+        c->d_span = static_cast<unsigned long long *>(dalloc(c, sizeof(unsigned long long) * 4 * kSpanSlots));
+        QX_CUDA(cudaMemsetAsync(c->d_span, 0, sizeof(unsigned long long) * 4 * kSpanSlots, c->stream));
+        c->h_span = static_cast<unsigned long long *>(halloc(c, sizeof(unsigned long long) * 4 * kSpanSlots));
+    }
+    DslashArgs a = a0;
+    const int slot = c->span_next;
+    c->span_next = (c->span_next + 1) % kSpanSlots;
+    a.span = c->d_span + 4 * slot;
     qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads, a.nrhs > 1 ? a.nrhs : 1,
-                           a.red_kind, c->cap_iter};
+                           a.red_kind, c->cap_iter, slot};
     if (c->capturing) {  // graph: external event-record nodes, re-recorded at each replay
         QX_CUDA(cudaEventRecordWithFlags(r.a, c->stream, cudaEventRecordExternal));
         launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
@@ -361,6 +371,16 @@ static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int
     launch_dslash_raw(prec, recon, dagger, kind, a, c->stream);
     QX_CUDA(cudaEventRecord(r.b, c->stream));
     c->trecs.push_back(r);
+}
+// host copy of the span slots (after a synchronisation); ms of one record's span
+static void fetch_spans(qudax_ctx *c) {
+    if (c->d_span) QX_CUDA(cudaMemcpy(c->h_span, c->d_span, sizeof(unsigned long long) * 4 * kSpanSlots,
+                                      cudaMemcpyDeviceToHost));
+}
+static double span_ms(const qudax_ctx *c, const qudax_ctx::TimingRec &r) {
+    if (r.span < 0 || !c->h_span) return 0.0;
+    const unsigned long long t0 = c->h_span[4 * r.span], t1 = c->h_span[4 * r.span + 1];
+    return t1 > t0 ? (double)(t1 - t0) * 1e-6 : 0.0;
 }
 
 // totals of one recorded launch: flops and bytes over its sites and right-hand sides (links and
@@ -385,6 +405,7 @@ static std::map<std::tuple<int, int, int>, std::pair<long, double>> g_tbreak;
 // the timing records of one replay of a captured graph (only those of the first `iters` solver
 // iterations of the batch: the later ones were halted and ran no work)
 void harvest_graph_timing(qudax_ctx *c, const std::vector<qudax_ctx::TimingRec> &recs, int iters) {
+    if (!recs.empty()) fetch_spans(c);
     for (auto &r : recs) {
         if (r.iter >= iters) continue;
         float ms = 0;
@@ -400,6 +421,7 @@ void harvest_graph_timing(qudax_ctx *c, const std::vector<qudax_ctx::TimingRec> 
         t.launches += 1;
         t.sites += r.sites * r.nrhs;
         t.ms += ms;
+        t.span_ms += span_ms(c, r);
         t.flops += m.flops;
         t.bytes_c += m.bytes_compulsory;
         t.bytes_p += m.bytes_paper;
@@ -1524,6 +1546,7 @@ qudax_status qudax_get_kernel_stats(qudax_ctx *c, int prec_filter, qudax_kernel_
     return guard(c, [&] {
         QX_CUDA(cudaStreamSynchronize(c->stream));
         std::memset(o, 0, sizeof(*o));
+        fetch_spans(c);
         for (auto &r : c->trecs) {
             if (prec_filter && r.prec != prec_filter) continue;
             float ms = 0;
@@ -1532,6 +1555,7 @@ qudax_status qudax_get_kernel_stats(qudax_ctx *c, int prec_filter, qudax_kernel_
             rec_model(r, &m);
             o->launches += 1;
             o->ms_total += ms;
+            o->span_ms_total += span_ms(c, r);
             o->sites += r.sites * r.nrhs;
             o->flops += m.flops;
             o->bytes_compulsory += m.bytes_compulsory;
@@ -1544,6 +1568,7 @@ qudax_status qudax_get_kernel_stats(qudax_ctx *c, int prec_filter, qudax_kernel_
             o->launches += t.launches;
             o->sites += t.sites;
             o->ms_total += t.ms;
+            o->span_ms_total += t.span_ms;
             o->flops += t.flops;
             o->bytes_compulsory += t.bytes_c;
             o->bytes_paper += t.bytes_p;

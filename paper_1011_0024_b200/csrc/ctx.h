@@ -39,6 +39,7 @@ struct qudax_ctx {
         int nrhs = 1;  // multi-RHS launch: links and clover are compulsory once, spinors per RHS
         int red = 0;   // fused reduction kind (RED_RHAT_DOT reads rhat: +1 spinor per site)
         int iter = 0;  // graph-captured launches: solver iteration within the batch
+        int span = -1; // slot of the launch's in-kernel span (first-CTA start, last-CTA end)
     };
     std::vector<TimingRec> trecs;
     std::vector<cudaEvent_t> ev_pool;
@@ -57,8 +58,11 @@ struct qudax_ctx {
     long long gauge_epoch = 0;
     struct TimingAcc {
         long long launches = 0, sites = 0;
-        double ms = 0, flops = 0, bytes_c = 0, bytes_p = 0;
+        double ms = 0, flops = 0, bytes_c = 0, bytes_p = 0, span_ms = 0;
     } tacc[3];
+    // in-kernel spans of the timed launches (device slots of 4 u64, host copy for harvesting)
+    unsigned long long *d_span = nullptr, *h_span = nullptr;
+    int span_next = 0;
     bool capturing = false;
     int cap_iter = 0;           // solver iteration (within the captured batch) being captured
     int flags = 0;              // qudax_init_flag bits

@@ -912,8 +912,41 @@ __device__ __forceinline__ int p2p_wait(const DslashArgs &a) {
     return (int)(s_seq & 1u);
 }
 
+// Kernel-timing span (kernel timing on: a.span != nullptr): the first CTA to arrive stamps
+// %globaltimer into span[0], the last CTA to finish into span[1] and resets the arrival counters
+// (span[2]: two 32-bit counters), so a launch slot can be replayed in a CUDA graph.  The span is
+// the kernel's own execution time, without the launch bubbles the event-record nodes around it
+// add in graph replay.  Not inlined: inlined, they cost the clover-inverse kernel 16 B of spills.
+__device__ __forceinline__ unsigned long long globaltimer_ns() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    return t;
+}
+__device__ __noinline__ void span_begin(unsigned long long *span) {
+    if (span && threadIdx.x == 0 && atomicAdd(reinterpret_cast<unsigned *>(span + 2), 1u) == 0u)
+        span[0] = globaltimer_ns();
+}
+__device__ __noinline__ void span_end(unsigned long long *span) {
+    if (!span) return;
+    // (thread 0's own end stands for its CTA's: no barrier, which would keep values live)
+    if (threadIdx.x == 0) {
+        if (atomicAdd(reinterpret_cast<unsigned *>(span + 2) + 1, 1u) == gridDim.x - 1) {
+            span[1] = globaltimer_ns();
+            span[2] = 0ull;  // both counters
+        }
+    }
+}
+
+template <int P, int RECON, bool DAG, int KIND, bool SS>
+__device__ __forceinline__ void dslash_body(const DslashArgs &a);
 template <int P, int RECON, bool DAG, int KIND, bool SS>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
+    span_begin(a.span);
+    dslash_body<P, RECON, DAG, KIND, SS>(a);
+    span_end(a.span);
+}
+template <int P, int RECON, bool DAG, int KIND, bool SS>
+__device__ __forceinline__ void dslash_body(const DslashArgs &a) {
     // one thread per output site (a one-wave grid-stride variant measured 8-25% slower: the
     // hardware CTA scheduler balances the memory-latency-bound CTAs better than a fixed wave)
     // multi-RHS (a.nrhs > 1): consecutive CTAs take the same sites for different right-hand

@@ -309,7 +309,15 @@ __device__ __forceinline__ void dslash_site_mr(const DslashArgs &a, int tid, int
 
 // grid: (site blocks) x (RHS groups of NR), consecutive CTAs = the groups of one site block
 template <int P, int RECON, bool DAG, int KIND, int NR>
+__device__ __forceinline__ void dslash_mr_body(const DslashArgs &a);
+template <int P, int RECON, bool DAG, int KIND, int NR>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, DslashMrMinBlocks<P, NR>::value) dslash_mr_kernel(const __grid_constant__ DslashArgs a) {
+    span_begin(a.span);
+    dslash_mr_body<P, RECON, DAG, KIND, NR>(a);
+    span_end(a.span);
+}
+template <int P, int RECON, bool DAG, int KIND, int NR>
+__device__ __forceinline__ void dslash_mr_body(const DslashArgs &a) {
     if (halted(a.halt)) return;
     const int ng = (a.nrhs + NR - 1) / NR;
     const int grp = blockIdx.x % ng, blk = blockIdx.x / ng;

@@ -220,6 +220,7 @@ struct DslashArgs {
     const int *halt;       // solver batch gate (SolverScalars::halt), nullptr outside solver batches
     int *err;              // device error word (kernel-initiated halo wait timeout -> QUDAX_ERR_COMM)
     int variant;           // kVariant* bits (init flags: test / comparison instantiations)
+    unsigned long long *span; // kernel timing on: {first-CTA start, last-CTA end, counters} (ns)
     // multi-RHS launch: nrhs > 1 uses in_m / out_m / x_m instead of in/out/x
     int nrhs;
     const void *in_m[kMaxRhs];

@@ -82,7 +82,8 @@ class SiteModel(ctypes.Structure):
 
 class KernelStats(ctypes.Structure):
     _fields_ = [("launches", ctypes.c_longlong), ("sites", ctypes.c_longlong), ("ms_total", ctypes.c_double),
-                ("flops", ctypes.c_double), ("bytes_compulsory", ctypes.c_double), ("bytes_paper", ctypes.c_double)]
+                ("flops", ctypes.c_double), ("bytes_compulsory", ctypes.c_double), ("bytes_paper", ctypes.c_double),
+                ("span_ms_total", ctypes.c_double)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}
