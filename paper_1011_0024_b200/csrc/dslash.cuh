@@ -922,11 +922,11 @@ __device__ __forceinline__ unsigned long long globaltimer_ns() {
     asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
     return t;
 }
-__device__ __noinline__ void span_begin(unsigned long long *span) {
+static __device__ __noinline__ void span_begin(unsigned long long *span) {
     if (span && threadIdx.x == 0 && atomicAdd(reinterpret_cast<unsigned *>(span + 2), 1u) == 0u)
         span[0] = globaltimer_ns();
 }
-__device__ __noinline__ void span_end(unsigned long long *span) {
+static __device__ __noinline__ void span_end(unsigned long long *span) {
     if (!span) return;
     // (thread 0's own end stands for its CTA's: no barrier, which would keep values live)
     if (threadIdx.x == 0) {
