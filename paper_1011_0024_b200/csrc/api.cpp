@@ -498,7 +498,13 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     args.in = in; args.out = out; args.x = x;
     int red_blocks = 0;  // CTA slots used in c->dpart by this call's launches
     const long n_int = g.n_int, n_bnd = g.Vh - g.n_int;
-    const bool split = c->comm == QUDAX_COMM_NCCL && !c->p2p.on && c->overlap && n_int > 0;
+    // NCCL path with overlap: ONE launch whose boundary CTAs (the grid's tail) wait for a flag the
+    // comm stream raises after the exchange (tail mode: no separate boundary launch, which ran at
+    // a fraction of a wave — 17 us for 1/16 of the sites at 32^3x64, gpurun r02e timeline), or,
+    // where the tail layout does not apply (the multi-RHS path), interior + boundary launches
+    const bool nccl_ov = c->comm == QUDAX_COMM_NCCL && !c->p2p.on && c->overlap && n_int > 0;
+    const bool tail_mode = nccl_ov && (spatial_split(g) ? true : g.T_loc > 2);
+    const bool split = nccl_ov && !tail_mode;
     const bool multi = sums_after_kernel(c);  // sums go through the transport before the recurrence
     if (red) {
         QX_CHECK(red->kind != RED_XDOT_NORM || kind >= QUDAX_CLOVER_XPAY, QUDAX_ERR_ARG, "x-dot needs xpay");
@@ -642,8 +648,33 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         mark(2, c->comm_stream);
         exchange_all(c, xf, nx, c->comm_stream);
         mark(3, c->comm_stream);
+        if (tail_mode) {
+            if (!c->tflags) {
+                c->tflags = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * 16));
+                QX_CUDA(cudaMemsetAsync(c->tflags, 0, sizeof(unsigned) * 16, c->stream));
+            }
+            launch_raise_flags(c->tflags, c->tflags + 8, g.split, c->halt, c->comm_stream);
+            c->launches += 1;
+        }
         QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
-        if (split) {
+        if (tail_mode) {
+            args.p2p_flags = c->tflags;
+            args.p2p_cseq = c->tflags + 9;
+            args.p2p_ccount = c->tflags + 10;
+            args.p2p_mask = g.split;
+            args.p2p_pdist = 0;
+            for (int m = 0; m < 3; ++m) args.sp2p_pdist[m] = 0;
+            args.reverse = 0;  // the waiting CTAs must be the last ones
+            args.tail_ni = spatial_split(g) ? (int)n_int : (int)((g.T_loc - 2) * g.F);
+            mark(4, c->stream);
+            launch(RANGE_TAIL, (int)g.Vh);
+            mark(5, c->stream);
+            mark(6, c->stream);
+            mark(7, c->stream);
+            // the join keeps the comm stream's next pack behind this Dslash (it overwrites the
+            // send buffers only after the ghosts of this one were consumed: ev_in of the next call)
+            QX_CUDA(cudaStreamWaitEvent(c->stream, c->ev_halo, 0));
+        } else if (split) {
             mark(4, c->stream);
             launch(RANGE_INTERIOR, (int)n_int);
             mark(5, c->stream);
@@ -1418,10 +1449,9 @@ qudax_status qudax_init(qudax_ctx **out, const qudax_init_param *p) {
             std::memcpy(&id, p->nccl_id, sizeof(id));
             QX_NCCL(ncclCommInitRank(&c->nccl, g.nranks, id, g.rank));
             // a second communicator for the global sums: the halo's send/recv run on the comm
-            // stream and the allreduces on the compute stream, and operations of ONE communicator
-            // issued from two streams may be serialised by NCCL in an order that deadlocks against
-            // the streams' own event dependencies (seen: the loopback solve with a Y/Z/T split
-            // hung once its sums went through NCCL)
+            // stream and the allreduces on the compute stream, so neither has to be ordered
+            // against the other inside one communicator (NCCL serialises a communicator's
+            // operations in issue order, whatever stream they were issued to)
             QX_NCCL(ncclCommSplit(c->nccl, 0, g.rank, &c->nccl_red, nullptr));
         }
         c->partials = static_cast<double *>(dalloc(c, sizeof(double) * 4 * blas_partial_blocks()));
@@ -1483,6 +1513,11 @@ qudax_status qudax_finalize(qudax_ctx *c) {
                          std::get<1>(kv.first), std::get<2>(kv.first), kv.second.first, 1e3 * kv.second.second / kv.second.first);
     if (c->stream) cudaStreamSynchronize(c->stream);
     if (c->comm_stream) cudaStreamSynchronize(c->comm_stream);
+    // the cached solver graphs first: graphs that captured NCCL operations hold references on
+    // the communicators (CUDA user objects), and ncclCommDestroy waits for them — with the graphs
+    // still alive it never returned (gpurun r02e: every NCCL-loopback solve test hung in close)
+    drop_graphs(c);  // (their timing events go back to the pool, destroyed below)
+    cudaDeviceSynchronize();  // lets the user objects' release callbacks run
     for (char *m : c->p2p.opened)
         if (m) cudaIpcCloseMemHandle(m);
     if (c->p2p.base) cudaFree(c->p2p.base);
@@ -1495,7 +1530,6 @@ qudax_status qudax_finalize(qudax_ctx *c) {
     for (void *p : c->host_allocs) cudaFreeHost(p);
     for (auto &r : c->trecs) { cudaEventDestroy(r.a); cudaEventDestroy(r.b); }
     for (auto &r : c->graph_trecs) { cudaEventDestroy(r.a); cudaEventDestroy(r.b); }
-    drop_graphs(c);  // (their timing events go back to the pool, destroyed below)
     for (auto e : c->ev_pool) cudaEventDestroy(e);
     for (auto e : c->xfer.done)
         if (e) cudaEventDestroy(e);

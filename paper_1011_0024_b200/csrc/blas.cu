@@ -54,6 +54,25 @@ void launch_coef(SolverScalars *S, int mode, const int *halt, cudaStream_t s) {
     QX_CUDA(cudaGetLastError());
 }
 
+// NCCL halo in tail mode (api.cpp dslash_op): after the exchange, one thread on the comm stream
+// advances this rank's producer sequence number and raises the flags of every split dimension;
+// the Dslash's boundary CTAs (RANGE_TAIL) acquire them (dslash.cuh p2p_wait).  A halted solver
+// batch skips it together with the consuming Dslash, so the two counters stay in step.
+__global__ void k_raise_flags(unsigned *flags, unsigned *seq, int mask, const int *halt) {
+    if (halted(halt)) return;
+    const unsigned s = *seq + 1u;
+    *seq = s;
+    for (int m = 0; m < 4; ++m) {
+        if (!(mask >> m & 1)) continue;
+        asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(flags + 2 * m), "r"(s) : "memory");
+        asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(flags + 2 * m + 1), "r"(s) : "memory");
+    }
+}
+void launch_raise_flags(unsigned *flags, unsigned *seq, int mask, const int *halt, cudaStream_t s) {
+    k_raise_flags<<<1, 1, 0, s>>>(flags, seq, mask, halt);
+    QX_CUDA(cudaGetLastError());
+}
+
 #define QX_GRID_LOOP(i) for (long i = (long)blockIdx.x * blockDim.x + threadIdx.x; i < Vh; i += (long)gridDim.x * blockDim.x)
 
 // p <- r + beta (p - omega v)            (BiCGstab search direction)

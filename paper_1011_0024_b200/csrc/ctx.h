@@ -110,6 +110,8 @@ struct qudax_ctx {
         void *mh_sb = nullptr, *mh_sf = nullptr, *mh_gb = nullptr, *mh_gf = nullptr;
     } halo[3];
     int *blist = nullptr;  // boundary sites (complement of the interior box) when X/Y/Z is split
+    // NCCL halo in tail mode: flags[4][2], producer seq, consumer seq, consumer CTA counter (device)
+    unsigned *tflags = nullptr;
 
     // kernel-initiated halo over peer memory (QUDAX_HALO_P2P).  One cudaMalloc region per rank,
     // identical layout on every rank: per precision and split dimension mu ghost_back[2],

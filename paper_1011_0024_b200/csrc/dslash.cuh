@@ -491,24 +491,6 @@ __device__ __forceinline__ void pf_spinor_l1(const void *base, long stride, long
         for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + j)));
     }
 }
-#ifndef QX_RED_STAGE
-#define QX_RED_STAGE 1
-#endif
-// 16-byte global -> shared copy that bypasses the registers (and L1: .cg)
-__device__ __forceinline__ void cp_async16(float4 *smem, const float4 *gmem) {
-    const unsigned sa = (unsigned)__cvta_generic_to_shared(smem);
-    asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa), "l"(gmem) : "memory");
-}
-__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
-__device__ __forceinline__ void cp_async_wait_all() { asm volatile("cp.async.wait_all;" ::: "memory"); }
-// this thread's staged 24 reals ([6][threads] float4 layout: conflict-free 16-byte accesses)
-__device__ __forceinline__ void stage_read(const float4 *stage, float *v) {
-#pragma unroll
-    for (int k = 0; k < 6; ++k) {
-        const float4 q = stage[k * QX_DSLASH_THREADS + threadIdx.x];
-        v[4 * k] = q.x; v[4 * k + 1] = q.y; v[4 * k + 2] = q.z; v[4 * k + 3] = q.w;
-    }
-}
 // one output site; red[] receives this site's contribution to the optional fused reduction
 // INMODE: load mode of the neighbour spinors (0 read-only path; 2 L2-coherent, for inputs
 // written by other CTAs earlier in the same launch — the fused Mhat kernel)
@@ -564,39 +546,10 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // accumulator as (1/a) T x, so its loads (x, clover) overlap the stencil's instead of
     // adding a dependent memory round trip after it; out = a * acc at the end.
     const bool xpay_early = (KIND == QUDAX_CLOVER_XPAY) && (a.a != 0.0);
-    // fp32 xpay kernels with a fused reduction: the reduction's second operand (x for
-    // (<out, x>, |out|^2), rhat0 for <rhat0, out>) is copied into shared memory by cp.async
-    // when the thread starts (no registers held, no L1 eviction risk), and read back from there
-    // after the store — the epilogue's dependent global round trip leaves every thread's tail
-    // (QX_RED_STAGE, fp32 only; 12 KB of shared memory per 128-thread CTA)
-    constexpr bool STAGE = QX_RED_STAGE && (P == 4) && (KIND == QUDAX_CLOVER_XPAY);
-    const bool staged = STAGE && a.red_kind != RED_NONE;
-    float4 *stage = nullptr;
-    if constexpr (STAGE) {
-        __shared__ float4 red_stage[6 * QX_DSLASH_THREADS];
-        stage = red_stage;
-        if (staged) {
-            const void *w = a.red_kind == RED_XDOT_NORM ? fx : (a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat);
-#pragma unroll
-            for (int k = 0; k < 6; ++k)
-                cp_async16(stage + k * QX_DSLASH_THREADS + threadIdx.x,
-                           reinterpret_cast<const float4 *>(w) + (long)k * a.stride + i);
-            cp_async_commit();
-        }
-    }
     if (xpay_early) {
         R v[24];
         Cx<R> xs[4][3];
-        if constexpr (STAGE) {
-            if (staged && a.red_kind == RED_XDOT_NORM) {  // x is in shared memory already
-                cp_async_wait_all();
-                stage_read(stage, v);
-            } else {
-                SpinorIO<P>::load(fx, a.stride, i, v);
-            }
-        } else {
-            SpinorIO<P>::load(fx, a.stride, i, v);
-        }
+        SpinorIO<P>::load(fx, a.stride, i, v);
         unpack_spinor(v, xs);
         apply_clover<P>(a.clover, a.stride, i, xs, acc);
         const R inv_a = (R)(1.0 / a.a);
@@ -850,14 +803,9 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // fused BiCGstab reductions over what was stored (half: the requantised values)
     SpinorIO<P>::store_requant(fout, a.stride, i, o);
     R w[24];
-    if constexpr (STAGE) {
-        cp_async_wait_all();
-        stage_read(stage, reinterpret_cast<float *>(w));
-    } else {
-        // (multi-RHS launch: this CTA's right-hand side, recomputed here rather than kept live)
-        const void *rh = a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat;
-        SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx : rh, a.stride, i, w);
-    }
+    // (multi-RHS launch: this CTA's right-hand side, recomputed here rather than kept live)
+    const void *rh = a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat;
+    SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx : rh, a.stride, i, w);
 #ifdef QX_RED_SITE_F64
     using RA = double;
 #else

@@ -327,6 +327,8 @@ __device__ __forceinline__ bool halted(const int *halt) {
 }
 #endif
 void launch_coef(SolverScalars *S, int mode, const int *halt, cudaStream_t s);
+// flags[2 mu], flags[2 mu + 1] = ++*seq for every mu in mask (NCCL halo tail mode)
+void launch_raise_flags(unsigned *flags, unsigned *seq, int mask, const int *halt, cudaStream_t s);
 void blas_xpy_mixed(int pd, int ps, const Geom &g, const void *x, void *y, cudaStream_t s);
 int blas_partial_blocks();
 
