@@ -699,7 +699,9 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     finish_red();
 }
 
-static void *tmp_odd(qudax_ctx *c, int prec) {
+void *tmp_odd_field(qudax_ctx *c, int prec);
+static void *tmp_odd(qudax_ctx *c, int prec) { return tmp_odd_field(c, prec); }
+void *tmp_odd_field(qudax_ctx *c, int prec) {
     auto &t = c->tmp_odd[prec_idx(prec)];
     if (!t) t = dalloc(c, spinor_bytes(prec, c->g.stride));
     return t;

@@ -165,6 +165,7 @@ inline int prec_idx(int prec) { return prec == 8 ? 0 : (prec == 4 ? 1 : 2); }
 void *dalloc(qudax_ctx *c, size_t bytes);
 void *halloc(qudax_ctx *c, size_t bytes);
 void dfree(qudax_ctx *c, void *p);  // releases a dalloc'ed buffer (no-op for nullptr)
+void *tmp_odd_field(qudax_ctx *c, int prec);  // the ctx's odd scratch field of precision prec
 void check_prec(int prec);
 // optional reduction fused into a Dslash epilogue (see DslashRed); res: 3 global sums (host)
 struct RedReq {

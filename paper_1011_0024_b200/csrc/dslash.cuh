@@ -491,9 +491,6 @@ __device__ __forceinline__ void pf_spinor_l1(const void *base, long stride, long
         for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + j)));
     }
 }
-#ifndef QX_LATE_XDOT
-#define QX_LATE_XDOT 1
-#endif
 // one output site; red[] receives this site's contribution to the optional fused reduction
 // INMODE: load mode of the neighbour spinors (0 read-only path; 2 L2-coherent, for inputs
 // written by other CTAs earlier in the same launch — the fused Mhat kernel)
@@ -548,11 +545,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // xpay: out = T x + a D in.  The site-local T x is computed FIRST and carried in the
     // accumulator as (1/a) T x, so its loads (x, clover) overlap the stencil's instead of
     // adding a dependent memory round trip after it; out = a * acc at the end.
-    // With the (<out, x>, |out|^2) reduction fused (the solver's t = Mhat s), T x is computed LATE
-    // instead (QX_LATE_XDOT): x is then loaded at the end for T x and re-read from L1 by the dot
-    // product right after, rather than early for T x and again from L2 after the store
-    const bool late_xdot = QX_LATE_XDOT && (KIND == QUDAX_CLOVER_XPAY) && (a.red_kind == RED_XDOT_NORM);
-    const bool xpay_early = (KIND == QUDAX_CLOVER_XPAY) && (a.a != 0.0) && !late_xdot;
+    const bool xpay_early = (KIND == QUDAX_CLOVER_XPAY) && (a.a != 0.0);
     if (xpay_early) {
         R v[24];
         Cx<R> xs[4][3];
@@ -788,19 +781,12 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
         for (int s = 0; s < 4; ++s)
 #pragma unroll
             for (int c = 0; c < 3; ++c) res[s][c] = co * acc[s][c];
-    } else {  // out = T x + a D in, T x computed last (a == 0, or the late-xdot form)
-        R xv[24];
+    } else {  // a == 0: out = T x
+        R v[24];
         Cx<R> xs[4][3];
-        SpinorIO<P>::load(fx, a.stride, i, xv);
-        unpack_spinor(xv, xs);
+        SpinorIO<P>::load(fx, a.stride, i, v);
+        unpack_spinor(v, xs);
         apply_clover<P>(a.clover, a.stride, i, xs, res);
-        if (late_xdot && a.a != 0.0) {
-            const R co = (R)a.a;
-#pragma unroll
-            for (int s = 0; s < 4; ++s)
-#pragma unroll
-                for (int c = 0; c < 3; ++c) res[s][c] = axpy(co, acc[s][c], res[s][c]);
-        }
     }
     R o[24];
 #pragma unroll
@@ -817,8 +803,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // fused BiCGstab reductions over what was stored (half: the requantised values)
     SpinorIO<P>::store_requant(fout, a.stride, i, o);
     R w[24];
-    // (multi-RHS launch: this CTA's right-hand side, recomputed here rather than kept live;
-    // late-xdot: x was just loaded for T x, so this re-read hits L1)
+    // (multi-RHS launch: this CTA's right-hand side, recomputed here rather than kept live)
     const void *rh = a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat;
     SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx : rh, a.stride, i, w);
 #ifdef QX_RED_SITE_F64

@@ -34,17 +34,33 @@ __device__ __forceinline__ Coord cb_coord(int i, int p, int X, int Y, int Z) {
 }
 
 // ============================================================================ spinors
+// The host-order slab holds one 192-byte DR record per site, sites of the two parities
+// interleaved; a parity field visits every other record.  Both directions stage a CTA's 128
+// records in shared memory so the global side moves whole records with consecutive 16-byte
+// accesses (one record per 12 lanes) — round 1's per-thread access of its own record (24 scalar
+// loads or stores 384 bytes apart across a warp) ran the export at ~1.1 TB/s (half-sector
+// writes; gpurun r01k launch list: 270 us per export at 32^3x64).
+constexpr int kXferThreads = 128;
 template <int P>
-__global__ void k_spinor_import(int X, int Y, int Z, int Vh, long stride, int parity, const double *__restrict__ src,
-                                void *__restrict__ dst) {
+__global__ void __launch_bounds__(kXferThreads) k_spinor_import(int X, int Y, int Z, int Vh, long stride, int parity,
+                                                                const double *__restrict__ src, void *__restrict__ dst) {
     using R = typename Prec<P>::R;
-    const int i = blockIdx.x * blockDim.x + threadIdx.x;
+    __shared__ double st[kXferThreads * 24];
+    __shared__ int lexs[kXferThreads];
+    const int i0 = blockIdx.x * kXferThreads;
+    const int i = i0 + threadIdx.x;
+    const int nsite = min(kXferThreads, Vh - i0);
+    if (i < Vh) lexs[threadIdx.x] = cb_coord(i, parity, X, Y, Z).lex;
+    __syncthreads();
+    for (int q = threadIdx.x; q < nsite * 12; q += kXferThreads) {
+        const int sidx = q / 12, ch = q - 12 * (q / 12);
+        const double2 v = __ldg(reinterpret_cast<const double2 *>(src + (size_t)lexs[sidx] * 24) + ch);
+        st[sidx * 24 + 2 * ch] = v.x;
+        st[sidx * 24 + 2 * ch + 1] = v.y;
+    }
+    __syncthreads();
     if (i >= Vh) return;
-    Coord c = cb_coord(i, parity, X, Y, Z);
-    const double *s = src + (size_t)c.lex * 24;
-    double d[24];
-#pragma unroll
-    for (int k = 0; k < 24; ++k) d[k] = s[k];
+    const double *d = st + threadIdx.x * 24;
     // psi_NR = S psi_DR: NR0 = (DR0 + DR2)/sqrt2, NR1 = (DR1 + DR3)/sqrt2,
     //                    NR2 = (DR0 - DR2)/sqrt2, NR3 = (DR1 - DR3)/sqrt2
     R o[24];
@@ -58,20 +74,31 @@ __global__ void k_spinor_import(int X, int Y, int Z, int Vh, long stride, int pa
 }
 
 template <int P>
-__global__ void k_spinor_export(int X, int Y, int Z, int Vh, long stride, int parity, const void *__restrict__ src,
-                                double *__restrict__ dst) {
+__global__ void __launch_bounds__(kXferThreads) k_spinor_export(int X, int Y, int Z, int Vh, long stride, int parity,
+                                                                const void *__restrict__ src, double *__restrict__ dst) {
     using R = typename Prec<P>::R;
-    const int i = blockIdx.x * blockDim.x + threadIdx.x;
-    if (i >= Vh) return;
-    Coord c = cb_coord(i, parity, X, Y, Z);
-    R v[24];
-    SpinorIO<P>::load(src, stride, i, v);
-    double *d = dst + (size_t)c.lex * 24;
+    __shared__ double st[kXferThreads * 24];
+    __shared__ int lexs[kXferThreads];
+    const int i0 = blockIdx.x * kXferThreads;
+    const int i = i0 + threadIdx.x;
+    const int nsite = min(kXferThreads, Vh - i0);
+    if (i < Vh) {
+        lexs[threadIdx.x] = cb_coord(i, parity, X, Y, Z).lex;
+        R v[24];
+        SpinorIO<P>::load(src, stride, i, v);
+        double *d = st + threadIdx.x * 24;
 #pragma unroll
-    for (int k = 0; k < 12; ++k) {
-        const double up = (double)v[k], lo = (double)v[k + 12];
-        d[k] = (up + lo) * kInvSqrt2;
-        d[k + 12] = (up - lo) * kInvSqrt2;
+        for (int k = 0; k < 12; ++k) {
+            const double up = (double)v[k], lo = (double)v[k + 12];
+            d[k] = (up + lo) * kInvSqrt2;
+            d[k + 12] = (up - lo) * kInvSqrt2;
+        }
+    }
+    __syncthreads();
+    for (int q = threadIdx.x; q < nsite * 12; q += kXferThreads) {
+        const int sidx = q / 12, ch = q - 12 * (q / 12);
+        reinterpret_cast<double2 *>(dst + (size_t)lexs[sidx] * 24)[ch] =
+            make_double2(st[sidx * 24 + 2 * ch], st[sidx * 24 + 2 * ch + 1]);
     }
 }
 
@@ -90,14 +117,14 @@ __global__ void k_spinor_convert(int Vh, long stride, void *__restrict__ dst, co
 static inline int nblk(long n, int t) { return (int)((n + t - 1) / t); }
 
 void launch_spinor_import(int prec, const Geom &g, int parity, const double *src, void *dst, cudaStream_t s) {
-    const int T = 128;
+    const int T = kXferThreads;
     if (prec == 8) k_spinor_import<8><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
     else if (prec == 4) k_spinor_import<4><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
     else k_spinor_import<2><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
     QX_CUDA(cudaGetLastError());
 }
 void launch_spinor_export(int prec, const Geom &g, int parity, const void *src, double *dst, cudaStream_t s) {
-    const int T = 128;
+    const int T = kXferThreads;
     if (prec == 8) k_spinor_export<8><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
     else if (prec == 4) k_spinor_export<4><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
     else k_spinor_export<2><<<nblk(g.Vh, T), T, 0, s>>>(g.X, g.Y, g.Z, (int)g.Vh, g.stride, parity, src, dst);
