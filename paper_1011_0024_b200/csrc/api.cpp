@@ -713,6 +713,9 @@ static void *tmp_even(qudax_ctx *c, int prec) {
 }
 
 // Mhat = T_ee - kappa^2 D_eo T_oo^{-1} D_oe (asymmetric Schur form on even sites)
+#ifndef QX_MATPC_REVERSE
+#define QX_MATPC_REVERSE 1
+#endif
 // symmetric Schur form: T_ee^{-1} Mhat.  Non-dagger: CLOVER_INV on odd,
 // CLOVER_INV_XPAY on even (fused reductions as for Mhat).  Dagger (explicit adjoint, not
 // gamma5-Hermitian): T_ee^{-1} in -> CLOVER_INV^dag on odd -> HOP^dag on even -> in - kappa^2 (.)
@@ -745,7 +748,7 @@ void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, con
     dslash_op(c, t, in, nullptr, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, nullptr);
     // the second kernel walks the lattice top-down: the timeslices the first kernel touched
     // last (their links, T^{-1} D in and the dirty tmp lines) are still in the 126 MB L2
-    dslash_op(c, out, t, in, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, red, 1);
+    dslash_op(c, out, t, in, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, red, QX_MATPC_REVERSE);
 }
 
 // Multi-RHS Dslash (SURVEY NEXT row 2, P:748-753 / P:1092-1094: many right-hand sides per
