@@ -276,7 +276,10 @@ qudax_status qudax_sync(qudax_ctx *ctx);
 /* Number of library kernels launched by this ctx so far (for launch accounting). */
 long long qudax_launch_count(const qudax_ctx *ctx);
 qudax_status qudax_get_partition(const qudax_ctx *ctx, qudax_partition *out);
-/* Enable (1) / disable (0) per-launch event timing of the Dslash kernels; clears the records. */
+/* Per-launch timing of the Dslash kernels; clears the records.  enable: 0 off; 1 CUDA events
+ * around every launch on the launching stream; 2 events plus the in-kernel span (first CTA's
+ * start to last CTA's end by %globaltimer, qudax_kernel_stats.span_ms_total), which costs the
+ * kernels a few microseconds of their own. */
 qudax_status qudax_kernel_timing(qudax_ctx *ctx, int enable);
 /* Synchronise and sum the recorded Dslash launches of precision prec_filter (0 = all). */
 qudax_status qudax_get_kernel_stats(qudax_ctx *ctx, int prec_filter, qudax_kernel_stats *out);

@@ -355,9 +355,12 @@ static void launch_dslash_ctx(qudax_ctx *c, int prec, int recon, int dagger, int
         c->h_span = static_cast<unsigned long long *>(halloc(c, sizeof(unsigned long long) * 4 * kSpanSlots));
     }
     DslashArgs a = a0;
-    const int slot = c->span_next;
-    c->span_next = (c->span_next + 1) % kSpanSlots;
-    a.span = c->d_span + 4 * slot;
+    int slot = -1;
+    if (c->timing == 2) {  // span mode: the kernels stamp their own start / end (a few us each)
+        slot = c->span_next;
+        c->span_next = (c->span_next + 1) % kSpanSlots;
+        a.span = c->d_span + 4 * slot;
+    }
     qudax_ctx::TimingRec r{pool_event(c), pool_event(c), prec, recon, kind, (long)a.nthreads, a.nrhs > 1 ? a.nrhs : 1,
                            a.red_kind, c->cap_iter, slot};
     if (c->capturing) {  // graph: external event-record nodes, re-recorded at each replay
@@ -1576,7 +1579,7 @@ qudax_status qudax_kernel_timing(qudax_ctx *c, int enable) {
         }
         c->trecs.clear();
         for (auto &t : c->tacc) t = qudax_ctx::TimingAcc{};
-        c->timing = enable != 0;
+        c->timing = enable == 2 ? 2 : (enable != 0 ? 1 : 0);
     });
 }
 

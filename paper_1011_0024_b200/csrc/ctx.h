@@ -31,7 +31,7 @@ struct qudax_ctx {
     bool sticky = false;
     long long launches = 0;
     // optional per-launch CUDA-event timing of the Dslash kernels (qudax_kernel_timing)
-    bool timing = false;
+    int timing = 0;  // 0 off, 1 CUDA events per Dslash launch, 2 events + in-kernel span
     struct TimingRec {
         cudaEvent_t a, b;
         int prec, recon, kind;

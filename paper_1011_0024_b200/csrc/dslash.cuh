@@ -688,14 +688,15 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             spatial_hop<MU, SB, true, DF>(ps, u, acc, sc);
         }
     };
-    // neighbour checkerboard indices of the six spatial hops (periodic wrap inside the box)
-    const int nxf = (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1, nxb = (x == 0 ? lex + (X - 1) : lex - 1) >> 1;
-    const int nyf = (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1, nyb = (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1;
-    const int nzf = (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1, nzb = (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1;
-    spatial(std::integral_constant<int, 0>{}, x, X, nxf, nxb);
+    // (neighbour indices computed at each call: holding all six live across the hops costs
+    // registers at the 80-register cap — measured up to 13 % on fp32 recon-8, r02m)
+    spatial(std::integral_constant<int, 0>{}, x, X, (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1,
+            (x == 0 ? lex + (X - 1) : lex - 1) >> 1);
     if (bail) return;
-    spatial(std::integral_constant<int, 1>{}, y, Y, nyf, nyb);
-    spatial(std::integral_constant<int, 2>{}, z, Z, nzf, nzb);
+    spatial(std::integral_constant<int, 1>{}, y, Y, (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1,
+            (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1);
+    spatial(std::integral_constant<int, 2>{}, z, Z, (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1,
+            (z == 0 ? lex + (Z - 1) * XY : lex - XY) >> 1);
 
     // ---- t direction: diagonal projectors, 12 reals per neighbour (eq. (6))
     {
@@ -889,9 +890,14 @@ template <int P, int RECON, bool DAG, int KIND, bool SS>
 __device__ __forceinline__ void dslash_body(const DslashArgs &a);
 template <int P, int RECON, bool DAG, int KIND, bool SS>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
-    span_begin(a.span);
+#ifndef QX_SPAN
+#define QX_SPAN 1
+#endif
+    // (the test is on the parameter, outside the calls: no call at all unless kernel timing runs
+    // in span mode)
+    if (QX_SPAN && a.span) span_begin(a.span);
     dslash_body<P, RECON, DAG, KIND, SS>(a);
-    span_end(a.span);
+    if (QX_SPAN && a.span) span_end(a.span);
 }
 template <int P, int RECON, bool DAG, int KIND, bool SS>
 __device__ __forceinline__ void dslash_body(const DslashArgs &a) {
@@ -902,7 +908,9 @@ __device__ __forceinline__ void dslash_body(const DslashArgs &a) {
 #ifndef QX_HALT_LATE
 #define QX_HALT_LATE 1
 #endif
-#if QX_HALT_LATE
+#if defined(QX_NO_HALT)
+    const int hv = 0;  // (experiment builds only: no solver-batch gate)
+#elif QX_HALT_LATE
     // the rest of a solver batch after a reliable-update request does nothing: the flag is read
     // now and tested after the first hop's loads are issued (dslash_site)
     const int hv = a.halt ? *reinterpret_cast<const volatile int *>(a.halt) : 0;

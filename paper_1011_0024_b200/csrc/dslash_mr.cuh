@@ -312,9 +312,9 @@ template <int P, int RECON, bool DAG, int KIND, int NR>
 __device__ __forceinline__ void dslash_mr_body(const DslashArgs &a);
 template <int P, int RECON, bool DAG, int KIND, int NR>
 __global__ void __launch_bounds__(QX_DSLASH_THREADS, DslashMrMinBlocks<P, NR>::value) dslash_mr_kernel(const __grid_constant__ DslashArgs a) {
-    span_begin(a.span);
+    if (a.span) span_begin(a.span);
     dslash_mr_body<P, RECON, DAG, KIND, NR>(a);
-    span_end(a.span);
+    if (a.span) span_end(a.span);
 }
 template <int P, int RECON, bool DAG, int KIND, int NR>
 __device__ __forceinline__ void dslash_mr_body(const DslashArgs &a) {

@@ -385,8 +385,10 @@ class Context:
     def sync(self):
         self._check(lib().qudax_sync(self._h))
 
-    def kernel_timing(self, enable=True):
-        self._check(lib().qudax_kernel_timing(self._h, int(bool(enable))))
+    def kernel_timing(self, enable=True, span=False):
+        """Per-launch CUDA-event timing of the Dslash kernels (span=True: also the in-kernel
+        %globaltimer span, which costs the kernels a few microseconds)."""
+        self._check(lib().qudax_kernel_timing(self._h, 2 if (enable and span) else int(bool(enable))))
 
     def halo_timeline(self, enable=True, read=False):
         """Diagnostic halo-overlap timeline (NCCL path): enable recording; with read=True return

@@ -54,8 +54,7 @@ def main():
             ks = ctx.kernel_stats()
             ctx.kernel_timing(False)
             gbs = ks["bytes_compulsory"] / (ks["ms_total"] * 1e-3) * 1e-9
-            res[name] = {"us": 1e3 * ks["ms_total"] / ks["launches"], "span_us": 1e3 * ks["span_ms_total"] / ks["launches"],
-                         "GBs": round(gbs, 1),
+            res[name] = {"us": 1e3 * ks["ms_total"] / ks["launches"], "GBs": round(gbs, 1),
                          "frac": round(gbs / peak, 4), "GFLOPS": round(ks["flops"] / (ks["ms_total"] * 1e-3) * 1e-9, 1)}
         for n in [int(v) for v in args.nrhs.split(",") if v]:
             ins = [ctx.new_field(prec) for _ in range(n)]
