@@ -344,7 +344,10 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     // host synchronisation inside a batch), cached across solves.  Not with the host transport
     // (its hooks run on the host and synchronise), which polls after every iteration.
     const bool host_comm = (c->comm == QUDAX_COMM_HOST);
-    const bool use_graph = !host_comm && !(c->flags & QUDAX_FLAG_NO_GRAPHS);
+#ifndef QX_EAGER_TIMING
+#define QX_EAGER_TIMING 0
+#endif
+    const bool use_graph = !host_comm && !(c->flags & QUDAX_FLAG_NO_GRAPHS) && !(QX_EAGER_TIMING && c->timing);
     const int batch = host_comm ? 1 : poll;
     bool first = true;
 
