@@ -28,6 +28,7 @@ def main():
     ap.add_argument("--cases", default="f32-12,h-12,f64-18")
     ap.add_argument("--tag", default=os.environ.get("QUDAX_LIB", "default"))
     ap.add_argument("--nrhs", default="", help="comma list: also time multi-RHS Mhat for these counts")
+    ap.add_argument("--flags", type=int, default=0, help="qudax init flags (A/B of kernel variants)")
     args = ap.parse_args()
     dims = tuple(int(v) for v in args.dims.split(","))
     try:
@@ -37,7 +38,7 @@ def main():
         peak = 6650.0
     U = qgen.gauge(dims, 1005, eps=-1.0)
     psi = qgen.spinor(dims, 2005)
-    ctx = qudax.Context(dims)
+    ctx = qudax.Context(dims, flags=args.flags)
     for case in args.cases.split(","):
         prec, recon = CASES[case]
         ctx.gauge_load(U, 0.124, 1.0, prec=prec, recon=recon)
