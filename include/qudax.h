@@ -66,7 +66,7 @@
 extern "C" {
 #endif
 
-#define QUDAX_ABI_VERSION 4
+#define QUDAX_ABI_VERSION 5
 
 typedef enum {
     QUDAX_OK = 0,
@@ -200,11 +200,12 @@ typedef struct {
     double *res_history;         /* optional host array: ||r_k|| / ||bhat|| after iteration k (the
                                     iterated residual, replaced by the true one at reliable updates) */
     int history_cap;             /* capacity of res_history (0 = none) */
-    int poll_every;              /* BiCGstab: iterations enqueued (one CUDA graph) between host reads of
-                                    the device-side scalars, 1..64 (0 = 4).  Algorithm R's update rule is
-                                    evaluated on the device after every iteration; an iteration that
-                                    calls for a reliable update stops the rest of the batch (its kernels
-                                    return at once), so the iterates do not depend on poll_every. */
+    int poll_every;              /* BiCGstab: at most this many iterations between host reads of the
+                                    device-side scalars, 1..64 (0 = 16).  A batch is one CUDA graph whose
+                                    WHILE node repeats the iteration on the device; Algorithm R's update
+                                    rule is evaluated on the device after every iteration, and an
+                                    iteration that calls for a reliable update (or converges) ends the
+                                    batch, so the iterates do not depend on poll_every. */
 } qudax_solve_param;
 
 typedef struct {
@@ -215,6 +216,8 @@ typedef struct {
     double flops;                /* effective flops (P:755-758 convention, reading Q16) */
     double gflops;
     int restarts;                /* Krylov restarts after a (near) breakdown of the sloppy recurrences */
+    int host_polls;              /* host reads of the device-side solver scalars (BiCGstab: batches) */
+    int device_batches;          /* of those, batches the device looped over in one WHILE-node graph */
 } qudax_solve_stats;
 
 /* Per-site work and traffic model, for reporting and tests. */

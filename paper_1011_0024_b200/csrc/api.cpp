@@ -462,7 +462,6 @@ static DslashArgs base_args(qudax_ctx *c, const qudax_ctx::GaugeCopy &gc, int pr
     args.bc_back = (g.c[3] == 0) ? (double)c->t_bc : 1.0;
     args.a = a;
     args.reverse = reverse;
-    args.halt = c->halt;
     args.err = c->d_err;
     args.variant = ((c->flags & QUDAX_FLAG_FORCE_SS) ? kVariantForceSS : 0) |
                    ((c->flags & QUDAX_FLAG_ONE_RHS_PER_THREAD) ? kVariantOneRhsPerThread : 0);
@@ -575,7 +574,6 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
         }
         pk.seq = reinterpret_cast<unsigned *>(q.base + q.off_seq);
         pk.count = reinterpret_cast<unsigned *>(q.base + q.off_count);
-        pk.halt = c->halt;
         pk.half_back = dagger ? 0 : 1;  // non-dagger: lower spins go backward (reading Q15)
         pk.half_fwd = dagger ? 1 : 0;
         auto pack = [&](cudaStream_t st) {
@@ -628,11 +626,11 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
     if (g.split & 8) xf[nx++] = Xfer{3, h.sf, h.sb, h.gb, h.gf, h.bytes, h.h_sf, h.h_sb, h.h_gb, h.h_gf};
     auto pack_all = [&](cudaStream_t st) {
         if (g.split & 8) {
-            launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, c->halt, st);
+            launch_pack_faces(prec, dagger, g, in, h.sb, h.sf, st);
             c->launches += 1;
         }
         if (spatial_split(g)) {
-            launch_pack_spatial(prec, dagger, g, 1 - p, in, h.ssb, h.ssf, c->halt, st);
+            launch_pack_spatial(prec, dagger, g, 1 - p, in, h.ssb, h.ssf, st);
             c->launches += 1;
         }
     };
@@ -656,7 +654,7 @@ void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec,
                 c->tflags = static_cast<unsigned *>(dalloc(c, sizeof(unsigned) * 16));
                 QX_CUDA(cudaMemsetAsync(c->tflags, 0, sizeof(unsigned) * 16, c->stream));
             }
-            launch_raise_flags(c->tflags, c->tflags + 8, g.split, c->halt, c->comm_stream);
+            launch_raise_flags(c->tflags, c->tflags + 8, g.split, c->comm_stream);
             c->launches += 1;
         }
         QX_CUDA(cudaEventRecord(c->ev_halo, c->comm_stream));
@@ -849,7 +847,7 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
     auto pack_all = [&](cudaStream_t st) {
         for (int k = 0; k < n; ++k) {
             launch_pack_faces(prec, dagger, g, in[k], static_cast<char *>(h.m_sb) + k * h.m_stride,
-                              static_cast<char *>(h.m_sf) + k * h.m_stride, c->halt, st);
+                              static_cast<char *>(h.m_sf) + k * h.m_stride, st);
             c->launches += 1;
         }
     };
@@ -923,7 +921,7 @@ int blas_op(qudax_ctx *c, int op, int prec, void *const *f, const double *coef, 
         if (op == OP_P_UPDATE || op == OP_FINAL) co[1].v = make_double2(coef[2], coef[3]);
     }
     RedTail tail{c->partials, c->d_counter, 0, 0, c->red_out, nullptr, COEF_NONE, c->dar, 0};
-    int n = blas_run(op, prec, c->g, f, co, tail, c->halt, c->stream);
+    int n = blas_run(op, prec, c->g, f, co, tail, c->stream);
     c->launches += 1;
     if (n) global_sum(c, c->red_out, n, res);
     return n;
@@ -941,7 +939,7 @@ void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, in
         QX_CUDA(cudaMemcpyAsync(dev_vals, c->h_red, sizeof(double) * n, cudaMemcpyHostToDevice, c->stream));
     }
     if (mode != COEF_NONE) {
-        launch_coef(S, mode, c->halt, c->stream);
+        launch_coef(S, mode, c->stream);
         c->launches += 1;
     }
 }
@@ -951,7 +949,7 @@ void device_sum_coef(qudax_ctx *c, double *dev_vals, int n, SolverScalars *S, in
 void blas_op_dev(qudax_ctx *c, int op, int prec, void *const *f, const CoefArg *co, SolverScalars *S, int mode) {
     const bool multi = sums_after_kernel(c);
     RedTail tail{c->partials, c->d_counter, 0, 0, S->red, S, multi ? COEF_NONE : mode, c->dar, 0};
-    int n = blas_run(op, prec, c->g, f, co, tail, c->halt, c->stream);
+    int n = blas_run(op, prec, c->g, f, co, tail, c->stream);
     c->launches += 1;
     if (n && multi) device_sum_coef(c, S->red, n, S, mode);
 }

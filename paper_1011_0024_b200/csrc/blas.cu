@@ -46,20 +46,29 @@ __device__ __forceinline__ void block_reduce_store(double (&v)[NRED], const RedT
 }
 
 // BiCGstab scalar recurrence after a multi-rank allreduce of S->red (single thread)
-__global__ void k_coef(SolverScalars *S, int mode, const int *halt) {
-    if (!halted(halt)) apply_coef(S, mode);
+__global__ void k_coef(SolverScalars *S, int mode) {
+    apply_coef(S, mode);
 }
-void launch_coef(SolverScalars *S, int mode, const int *halt, cudaStream_t s) {
-    k_coef<<<1, 1, 0, s>>>(S, mode, halt);
+// first / last node of a batch graph (solver.cpp): the WHILE node's condition handle for the
+// reduction tail that evaluates Algorithm R, and the batch's last iteration
+__global__ void k_batch_begin(SolverScalars *S, unsigned long long cond, int n) {
+    S->cond = cond;
+    S->kstop = S->k + n;
+}
+__global__ void k_batch_end(SolverScalars *S) { S->cond = 0ull; }
+void launch_batch_begin(SolverScalars *S, unsigned long long cond, int n, cudaStream_t s) {
+    k_batch_begin<<<1, 1, 0, s>>>(S, cond, n);
+}
+void launch_batch_end(SolverScalars *S, cudaStream_t s) { k_batch_end<<<1, 1, 0, s>>>(S); }
+void launch_coef(SolverScalars *S, int mode, cudaStream_t s) {
+    k_coef<<<1, 1, 0, s>>>(S, mode);
     QX_CUDA(cudaGetLastError());
 }
 
 // NCCL halo in tail mode (api.cpp dslash_op): after the exchange, one thread on the comm stream
 // advances this rank's producer sequence number and raises the flags of every split dimension;
-// the Dslash's boundary CTAs (RANGE_TAIL) acquire them (dslash.cuh p2p_wait).  A halted solver
-// batch skips it together with the consuming Dslash, so the two counters stay in step.
-__global__ void k_raise_flags(unsigned *flags, unsigned *seq, int mask, const int *halt) {
-    if (halted(halt)) return;
+// the Dslash's boundary CTAs (RANGE_TAIL) acquire them (dslash.cuh p2p_wait).
+__global__ void k_raise_flags(unsigned *flags, unsigned *seq, int mask) {
     const unsigned s = *seq + 1u;
     *seq = s;
     for (int m = 0; m < 4; ++m) {
@@ -68,8 +77,8 @@ __global__ void k_raise_flags(unsigned *flags, unsigned *seq, int mask, const in
         asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(flags + 2 * m + 1), "r"(s) : "memory");
     }
 }
-void launch_raise_flags(unsigned *flags, unsigned *seq, int mask, const int *halt, cudaStream_t s) {
-    k_raise_flags<<<1, 1, 0, s>>>(flags, seq, mask, halt);
+void launch_raise_flags(unsigned *flags, unsigned *seq, int mask, cudaStream_t s) {
+    k_raise_flags<<<1, 1, 0, s>>>(flags, seq, mask);
     QX_CUDA(cudaGetLastError());
 }
 
@@ -77,9 +86,7 @@ void launch_raise_flags(unsigned *flags, unsigned *seq, int mask, const int *hal
 
 // p <- r + beta (p - omega v)            (BiCGstab search direction)
 template <int P>
-__global__ void k_p_update(long Vh, long stride, const void *r, void *p, const void *v, CoefArg beta_, CoefArg omega_,
-                           const int *halt) {
-    if (halted(halt)) return;
+__global__ void k_p_update(long Vh, long stride, const void *r, void *p, const void *v, CoefArg beta_, CoefArg omega_) {
     using R = typename Prec<P>::R;
     const double2 beta = coef_get(beta_), omega = coef_get(omega_);
     const Cx<R> b = cx((R)beta.x, (R)beta.y), w = cx((R)omega.x, (R)omega.y);
@@ -101,8 +108,7 @@ __global__ void k_p_update(long Vh, long stride, const void *r, void *p, const v
 
 // y <- y + c x   (c complex)
 template <int P>
-__global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y, const int *halt) {
-    if (halted(halt)) return;
+__global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y) {
     using R = typename Prec<P>::R;
     const double2 c = coef_get(c_);
     const Cx<R> a = cx((R)c.x, (R)c.y);
@@ -122,8 +128,7 @@ __global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y
 
 // z <- x + a y  (real a); z may alias x or y
 template <int P>
-__global__ void k_xpay(long Vh, long stride, const void *x, double a, const void *y, void *z, const int *halt) {
-    if (halted(halt)) return;
+__global__ void k_xpay(long Vh, long stride, const void *x, double a, const void *y, void *z) {
     using R = typename Prec<P>::R;
     QX_GRID_LOOP(i) {
         R xx[24], yy[24];
@@ -137,8 +142,7 @@ __global__ void k_xpay(long Vh, long stride, const void *x, double a, const void
 
 // sum conj(a) b -> (re, im)
 template <int P>
-__global__ void k_cdot(long Vh, long stride, const void *a, const void *b, RedTail tail, const int *halt) {
-    if (halted(halt)) return;
+__global__ void k_cdot(long Vh, long stride, const void *a, const void *b, RedTail tail) {
     using R = typename Prec<P>::R;
     double acc[2] = {0, 0};
     QX_GRID_LOOP(i) {
@@ -156,8 +160,7 @@ __global__ void k_cdot(long Vh, long stride, const void *a, const void *b, RedTa
 
 // sum |a|^2
 template <int P>
-__global__ void k_norm2(long Vh, long stride, const void *a, RedTail tail, const int *halt) {
-    if (halted(halt)) return;
+__global__ void k_norm2(long Vh, long stride, const void *a, RedTail tail) {
     using R = typename Prec<P>::R;
     double acc[1] = {0};
     QX_GRID_LOOP(i) {
@@ -171,8 +174,7 @@ __global__ void k_norm2(long Vh, long stride, const void *a, RedTail tail, const
 
 // (<t, s>, |t|^2)
 template <int P>
-__global__ void k_tdot(long Vh, long stride, const void *t, const void *s, RedTail tail, const int *halt) {
-    if (halted(halt)) return;
+__global__ void k_tdot(long Vh, long stride, const void *t, const void *s, RedTail tail) {
     using R = typename Prec<P>::R;
     double acc[3] = {0, 0, 0};
     QX_GRID_LOOP(i) {
@@ -196,8 +198,7 @@ __global__ void k_tdot(long Vh, long stride, const void *t, const void *s, RedTa
 template <int P>
 __global__ void __launch_bounds__(kBlasThreads, P == 4 ? QX_BICG_MINB : 1)
 k_bicg_final(long Vh, long stride, void *x, const void *p, void *s, const void *t, const void *rhat,
-                             CoefArg alpha_, CoefArg omega_, RedTail tail, const int *halt) {
-    if (halted(halt)) return;
+                             CoefArg alpha_, CoefArg omega_, RedTail tail) {
     using R = typename Prec<P>::R;
     const double2 alpha = coef_get(alpha_), omega = coef_get(omega_);
     const Cx<R> al = cx((R)alpha.x, (R)alpha.y), om = cx((R)omega.x, (R)omega.y);
@@ -295,8 +296,7 @@ __global__ void k_xpy_mixed(long Vh, long stride, const void *x, void *y) {
 
 // r <- b - r ; returns |r|^2
 template <int P>
-__global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, RedTail tail, const int *halt) {
-    if (halted(halt)) return;
+__global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, RedTail tail) {
     using R = typename Prec<P>::R;
     double acc[1] = {0};
     QX_GRID_LOOP(i) {
@@ -330,38 +330,38 @@ __global__ void k_bmr_norm(long Vh, long stride, const void *b, void *r, RedTail
         K<<<B_, kBlasThreads, 0, s>>>(__VA_ARGS__);    \
     } while (0)
 
-int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail, const int *halt,
+int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail,
              cudaStream_t s) {
     const long Vh = g.Vh, st = g.stride;
     int nred = 0;
     switch (op) {
         case OP_P_UPDATE:  // p = r + beta (p - omega v): r=f0, p=f1, v=f2
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_p_update<P>, Vh, st, f[0], f[1], f[2], co[0], co[1], halt));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_p_update<P>, Vh, st, f[0], f[1], f[2], co[0], co[1]));
             break;
         case OP_CAXPY:  // f1 += c f0
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_caxpy<P>, Vh, st, co[0], f[0], f[1], halt));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_caxpy<P>, Vh, st, co[0], f[0], f[1]));
             break;
         case OP_XPAY:  // f2 = f0 + a f1
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_xpay<P>, Vh, st, f[0], co[0].v.x, f[1], f[2], halt));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_xpay<P>, Vh, st, f[0], co[0].v.x, f[1], f[2]));
             break;
         case OP_CDOT:  // <f0, f1>
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_cdot<P>, Vh, st, f[0], f[1], tail, halt));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_cdot<P>, Vh, st, f[0], f[1], tail));
             nred = 2;
             break;
         case OP_NORM2:
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_norm2<P>, Vh, st, f[0], tail, halt));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_norm2<P>, Vh, st, f[0], tail));
             nred = 1;
             break;
         case OP_TDOT:  // (<f0, f1>, |f0|^2)
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_tdot<P>, Vh, st, f[0], f[1], tail, halt));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_tdot<P>, Vh, st, f[0], f[1], tail));
             nred = 3;
             break;
         case OP_FINAL:  // x=f0, p=f1, s=f2, t=f3, rhat=f4
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bicg_final<P>, Vh, st, f[0], f[1], f[2], f[3], f[4], co[0], co[1], tail, halt));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bicg_final<P>, Vh, st, f[0], f[1], f[2], f[3], f[4], co[0], co[1], tail));
             nred = 3;
             break;
         case OP_BMR_NORM:  // f1 = f0 - f1
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bmr_norm<P>, Vh, st, f[0], f[1], tail, halt));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_bmr_norm<P>, Vh, st, f[0], f[1], tail));
             nred = 1;
             break;
         default:

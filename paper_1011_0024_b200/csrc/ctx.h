@@ -51,7 +51,9 @@ struct qudax_ctx {
     struct Graph {
         std::vector<uintptr_t> key;
         cudaGraphExec_t exec = nullptr;
-        long long launches = 0;          // library kernels per replay
+        long long launches = 0;          // library kernels per replay (WHILE graphs: outside the loop)
+        long long per_iter = 0;          // WHILE graphs: library kernels per loop iteration
+        bool no_while = false;           // this key's iteration cannot sit in a WHILE node
         std::vector<TimingRec> trecs;    // event-bracketed Dslash launches (kernel timing on)
     };
     std::vector<Graph> graphs;
@@ -66,9 +68,6 @@ struct qudax_ctx {
     bool capturing = false;
     int cap_iter = 0;           // solver iteration (within the captured batch) being captured
     int flags = 0;              // qudax_init_flag bits
-    // solver batch gate: while set, every kernel the library launches carries this pointer
-    // (SolverScalars::halt) and returns at once when an earlier iteration set it
-    const int *halt = nullptr;
     // device error word in mapped pinned host memory (kernel-initiated halo wait timeout)
     int *h_err = nullptr, *d_err = nullptr;
     // the Schur form matpc_op applies: 0 asymmetric (default), 1 symmetric (set by a solve with

@@ -498,7 +498,7 @@ __device__ __forceinline__ void pf_spinor_l1(const void *base, long stride, long
 // separate instantiation so the unpartitioned kernels keep their register allocation
 template <int P, int RECON, bool DAG, int KIND, int INMODE = 0, bool SS = false>
 __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin, void *fout, const void *fx, int tid,
-                                            double red[3], long goff = 0, int sbit = 0, int hv = 0) {
+                                            double red[3], long goff = 0, int sbit = 0) {
     using R = typename Prec<P>::R;
     if (a.reverse) tid = a.nthreads - 1 - tid;
     const int X = a.X, Y = a.Y, Z = a.Z, Xh = a.Xh;
@@ -569,7 +569,6 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // flight per thread (dslash_pair).
     constexpr bool PAIR = dslash_pair<P, RECON>();
     constexpr bool DF = dslash_defer<P, RECON>();
-    bool bail = false;
     auto spatial = [&](auto mu_c, int coord, int Lmu, int nf, int nb) {
         constexpr int MU = decltype(mu_c)::value;
         // operand sources of the two hops: the input field, or (partitioned X) the neighbour's
@@ -642,15 +641,6 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
             sb.template load_spinor<INMODE>(bsrc, bstr, nb);
             lb.load(lbsrc, lbstr, lbi);
         }
-        if constexpr (MU == 0) {
-            // a halted solver batch (SolverScalars::halt): the flag was loaded at kernel entry and
-            // is tested only here, after the first hop's loads are in flight, so its latency is
-            // not added to every thread's critical path
-            if (hv) {
-                bail = true;
-                return;
-            }
-        }
         if constexpr (DF && QX_BPROJ) {
             R v[24];
             Cx<R> ps[4][3], u[3][3], h0[3], h1[3];
@@ -692,7 +682,6 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // registers at the 80-register cap — measured up to 13 % on fp32 recon-8, r02m)
     spatial(std::integral_constant<int, 0>{}, x, X, (x == X - 1 ? lex - (X - 1) : lex + 1) >> 1,
             (x == 0 ? lex + (X - 1) : lex - 1) >> 1);
-    if (bail) return;
     spatial(std::integral_constant<int, 1>{}, y, Y, (y == Y - 1 ? lex - (Y - 1) * X : lex + X) >> 1,
             (y == 0 ? lex + (Y - 1) * X : lex - X) >> 1);
     spatial(std::integral_constant<int, 2>{}, z, Z, (z == Z - 1 ? lex - (Z - 1) * XY : lex + XY) >> 1,
@@ -905,19 +894,8 @@ __device__ __forceinline__ void dslash_body(const DslashArgs &a) {
     // hardware CTA scheduler balances the memory-latency-bound CTAs better than a fixed wave)
     // multi-RHS (a.nrhs > 1): consecutive CTAs take the same sites for different right-hand
     // sides, so the links and clover they stream are served from L2 after the first of them
-#ifndef QX_HALT_LATE
-#define QX_HALT_LATE 1
-#endif
-#if defined(QX_NO_HALT)
-    const int hv = 0;  // (experiment builds only: no solver-batch gate)
-#elif QX_HALT_LATE
-    // the rest of a solver batch after a reliable-update request does nothing: the flag is read
-    // now and tested after the first hop's loads are issued (dslash_site)
-    const int hv = a.halt ? *reinterpret_cast<const volatile int *>(a.halt) : 0;
-#else
-    if (halted(a.halt)) return;
-    const int hv = 0;
-#endif
+    // (no solver-batch gate: a batch's remaining iterations after a reliable-update request are
+    // not launched at all — the WHILE node of the batch graph stops, solver.cpp)
     int blk = blockIdx.x, rhs = 0;
     if (a.nrhs > 1) {
         rhs = blk % a.nrhs;
@@ -932,12 +910,10 @@ __device__ __forceinline__ void dslash_body(const DslashArgs &a) {
     int sbit = 0;                               // kernel-initiated halo: sequence parity of the ghosts
     // RANGE_TAIL: only CTAs holding boundary sites (the grid's last ones) wait for the halo
     if (a.p2p_flags && (a.range != RANGE_TAIL || (blk + 1) * (int)blockDim.x > a.tail_ni)) {
-        if (hv) return;  // (the matching pack kernel was halted too: no flag to wait for)
         sbit = p2p_wait(a);
         goff = sbit ? a.p2p_pdist : 0L;
     }
-    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND, 0, SS>(a, fin, fout, fx, tid, red, goff, sbit, hv);
-    if (hv) return;
+    if (tid < a.nthreads) dslash_site<P, RECON, DAG, KIND, 0, SS>(a, fin, fout, fx, tid, red, goff, sbit);
     if (a.p2p_flags) {  // the last CTA to finish advances the consumed-halo counter
         __syncthreads();
         if (threadIdx.x == 0 && atomicAdd(a.p2p_ccount, 1u) == gridDim.x - 1) {

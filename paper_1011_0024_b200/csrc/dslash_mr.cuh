@@ -318,7 +318,6 @@ __global__ void __launch_bounds__(QX_DSLASH_THREADS, DslashMrMinBlocks<P, NR>::v
 }
 template <int P, int RECON, bool DAG, int KIND, int NR>
 __device__ __forceinline__ void dslash_mr_body(const DslashArgs &a) {
-    if (halted(a.halt)) return;
     const int ng = (a.nrhs + NR - 1) / NR;
     const int grp = blockIdx.x % ng, blk = blockIdx.x / ng;
     const int r0 = grp * NR;

@@ -83,10 +83,11 @@ inline int spatial_split(const Geom &g) { return g.split & 7; }
 // device-resident BiCGstab scalars (Algorithm R), advanced by apply_coef after each reduction
 // The iteration's update rule (Algorithm R, solver.cpp) is evaluated on the device right after
 // the |r|^2 reduction (COEF_RHO with decide != 0): the host reads the scalars once per batch of
-// `poll_every` iterations instead of after every iteration.  An iteration that calls for a
-// reliable update sets `halt`; every kernel launched for the rest of the batch (they carry a
-// pointer to it) returns at once, so the iterates are exactly those of a host decision taken
-// after every iteration.
+// up to `poll_every` iterations instead of after every iteration.  A batch is a CUDA graph whose
+// WHILE node repeats one iteration while the condition `cond` holds; the tail that evaluates
+// the rule clears it when the iteration calls for a reliable update (`halt`), converged, or
+// completes the batch (k == kstop) — so no further kernel of the batch is launched at all, and
+// the iterates are exactly those of a host decision taken after every iteration.
 constexpr int kHistRing = 64;  // per-iteration |r| of the current batch (poll_every <= kHistRing)
 struct SolverScalars {
     double2 rho, rho_new, alpha, malpha, omega, beta;
@@ -99,7 +100,8 @@ struct SolverScalars {
     int decide;                  // evaluate the update rule after COEF_RHO
     int halt;                    // an iteration of this batch asked for a reliable update
     int updX, blown;             // its flags (reading R3 for blown)
-    int pad_;
+    int kstop;                   // the batch's last iteration (WHILE-graph batches)
+    unsigned long long cond;     // cudaGraphConditionalHandle of the running batch graph, 0: none
     double hist[kHistRing];      // |r_k| (iterated) at ring slot (k - 1) % kHistRing
 };
 enum CoefMode { COEF_NONE = 0, COEF_ALPHA = 1, COEF_OMEGA = 2, COEF_RHO = 3 };
@@ -217,7 +219,6 @@ struct DslashArgs {
     RedTail tail;          // 3 sums per CTA; block_offset set per launch (split launches)
     const void *rhat;
     int reverse;           // 1: map CTAs to sites from the top of the range down (L2 reuse, see matpc)
-    const int *halt;       // solver batch gate (SolverScalars::halt), nullptr outside solver batches
     int *err;              // device error word (kernel-initiated halo wait timeout -> QUDAX_ERR_COMM)
     int variant;           // kVariant* bits (init flags: test / comparison instantiations)
     unsigned long long *span; // kernel timing on: {first-CTA start, last-CTA end, counters} (ns)
@@ -247,7 +248,7 @@ int dslash_blocks_f16(int recon, int dagger, int kind, int nthreads);
 // x_mu = 0 face projected with the receiver's forward-hop projector -> sb[mu], the x_mu = L-1
 // face with its backward-hop projector -> sf[mu]; 12 reals per site in the arithmetic precision
 void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, const void *in, void *const sb[3],
-                         void *const sf[3], const int *halt, cudaStream_t s);
+                         void *const sf[3], cudaStream_t s);
 // whether the faces along mu carry raw spinor records (half everywhere; X in every precision)
 // instead of spin-projected half spinors in the arithmetic precision
 __host__ __device__ inline bool sface_raw(int prec, int mu) { return prec == 2 || mu == 0; }
@@ -256,7 +257,7 @@ size_t sface_bytes(int prec, int mu, long fs);
 // face pack: t_loc = 0 slice half (lower if !dagger) -> send_back; t_loc = T_loc-1 half
 // (upper if !dagger) -> send_fwd.  `in` is the Dslash input field (parity 1-p).
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back,
-                       void *send_fwd, const int *halt, cudaStream_t s);
+                       void *send_fwd, cudaStream_t s);
 
 // kernel-initiated halo of any process grid (QUDAX_HALO_P2P): all split dimensions' faces
 // stored into the neighbours' ghosts (peer memory), then their flags raised (layout.cu)
@@ -272,7 +273,6 @@ struct P2PPackArgs {
     unsigned *flag_b[4];    // backward neighbour's "forward ghost filled" flag of mu
     unsigned *flag_f[4];    // forward neighbour's "backward ghost filled" flag of mu
     unsigned *seq, *count;  // this rank's producer sequence and CTA counter
-    const int *halt;
     int half_back, half_fwd; // T faces: spin halves sent backward / forward (reading Q15)
 };
 void launch_pack_p2p(int prec, int dagger, const P2PPackArgs &a, const void *in, cudaStream_t s);
@@ -317,18 +317,13 @@ __device__ __forceinline__ double2 coef_get(const CoefArg &c) { return c.d ? *c.
 #endif
 // `tail` describes the reduction of reducing ops (partials/counter/out/S/coef_mode; the
 // block fields are filled in here).  Returns the number of reduced doubles (0 if none).
-int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail, const int *halt,
+int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co, RedTail tail,
              cudaStream_t s);
-#ifdef __CUDACC__
-// a kernel launched inside a solver batch returns at once once an earlier iteration has asked
-// for a reliable update (SolverScalars::halt); halt == nullptr outside solver batches
-__device__ __forceinline__ bool halted(const int *halt) {
-    return halt && *reinterpret_cast<const volatile int *>(halt);
-}
-#endif
-void launch_coef(SolverScalars *S, int mode, const int *halt, cudaStream_t s);
+void launch_coef(SolverScalars *S, int mode, cudaStream_t s);
+void launch_batch_begin(SolverScalars *S, unsigned long long cond, int n, cudaStream_t s);
+void launch_batch_end(SolverScalars *S, cudaStream_t s);
 // flags[2 mu], flags[2 mu + 1] = ++*seq for every mu in mask (NCCL halo tail mode)
-void launch_raise_flags(unsigned *flags, unsigned *seq, int mask, const int *halt, cudaStream_t s);
+void launch_raise_flags(unsigned *flags, unsigned *seq, int mask, cudaStream_t s);
 void blas_xpy_mixed(int pd, int ps, const Geom &g, const void *x, void *y, cudaStream_t s);
 int blas_partial_blocks();
 

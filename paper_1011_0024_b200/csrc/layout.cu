@@ -613,8 +613,7 @@ __device__ __forceinline__ void k_pack_faces_body(long F, long T_loc, long strid
 }
 template <int P>
 __global__ void k_pack_faces(long F, long T_loc, long stride, long fstride, int half_back, int half_fwd,
-                             const void *__restrict__ in, void *__restrict__ sb, void *__restrict__ sf, const int *halt) {
-    if (halted(halt)) return;
+                             const void *__restrict__ in, void *__restrict__ sb, void *__restrict__ sf) {
     k_pack_faces_body<P>(F, T_loc, stride, fstride, half_back, half_fwd, in, sb, sf);
 }
 
@@ -642,7 +641,6 @@ struct SPackArgs {
     int q;          // parity of the packed (input) field
     long Fd[3], fsd[3], stride;
     void *sb[3], *sf[3];
-    const int *halt;
 };
 // one face site of a partitioned X / Y / Z (face index f of dimension mu, fwd: the x_mu = L-1
 // face) -> dst (face layout, fs padded sites)
@@ -689,7 +687,6 @@ __device__ __forceinline__ void pack_spatial_one(int mu, long f, bool fwd, const
 
 template <int P, bool DAG>
 __global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *__restrict__ in) {
-    if (halted(a.halt)) return;
     long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
     int mu = 0;
     for (; mu < 3; ++mu) {
@@ -711,7 +708,6 @@ __global__ void k_pack_spatial(const __grid_constant__ SPackArgs a, const void *
 template <int P, bool DAG>
 __global__ void k_pack_p2p(const __grid_constant__ P2PPackArgs a, const void *__restrict__ in) {
     __shared__ bool last;
-    if (halted(a.halt)) return;
     const unsigned s = *reinterpret_cast<volatile unsigned *>(a.seq) + 1u;
     const bool odd = (s & 1u) != 0;
     long k = (long)blockIdx.x * blockDim.x + threadIdx.x;
@@ -785,9 +781,8 @@ void launch_pack_p2p(int prec, int dagger, const P2PPackArgs &a, const void *in,
 size_t sface_bytes(int prec, int mu, long fs) { return sface_raw(prec, mu) ? spinor_bytes(prec, fs) : (size_t)12 * prec * fs; }
 
 void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, const void *in, void *const sb[3],
-                         void *const sf[3], const int *halt, cudaStream_t s) {
+                         void *const sf[3], cudaStream_t s) {
     SPackArgs a{};
-    a.halt = halt;
     long n = 0;
     for (int m = 0; m < 4; ++m) a.L[m] = g.L[m];
     a.mask = spatial_split(g);
@@ -816,7 +811,7 @@ void launch_pack_spatial(int prec, int dagger, const Geom &g, int in_parity, con
 }
 
 void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void *send_back, void *send_fwd,
-                       const int *halt, cudaStream_t s) {
+                       cudaStream_t s) {
     // non-dagger: the receiver's forward hop (1 - gamma_4) needs LOWER spins of our t=0 slice
     // (sent backward); its backward hop (1 + gamma_4) needs UPPER spins of our t=T_loc-1 slice
     // (sent forward).  The dagger swaps the halves (reading Q15).
@@ -824,9 +819,9 @@ void launch_pack_faces(int prec, int dagger, const Geom &g, const void *in, void
     const int half_fwd = dagger ? 1 : 0;
     const int T = 128;
     const int b = nblk(2 * g.F, T);
-    if (prec == 8) k_pack_faces<8><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd, halt);
-    else if (prec == 4) k_pack_faces<4><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd, halt);
-    else k_pack_faces<2><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd, halt);
+    if (prec == 8) k_pack_faces<8><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
+    else if (prec == 4) k_pack_faces<4><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
+    else k_pack_faces<2><<<b, T, 0, s>>>(g.F, g.T_loc, g.stride, g.fstride, half_back, half_fwd, in, send_back, send_fwd);
     QX_CUDA(cudaGetLastError());
 }
 

@@ -165,12 +165,106 @@ static qudax_ctx::Graph *cached_graph(qudax_ctx *c, std::vector<uintptr_t> key, 
     return &c->graphs.back();
 }
 
-// RAII: kernels launched while this is alive carry the solver batch gate
-struct HaltGate {
-    qudax_ctx *c;
-    HaltGate(qudax_ctx *c_, const int *h) : c(c_) { c->halt = h; }
-    ~HaltGate() { c->halt = nullptr; }
-};
+// Batch graph (solve_dev): [k_batch_begin] -> WHILE(cond) { one iteration } -> [k_batch_end].
+// The WHILE node repeats the captured iteration on the device until the reduction tail that
+// evaluates Algorithm R clears the condition (reliable update, convergence, maxiter, or the
+// batch's `n` iterations done): no host round trip and no launch inside a batch, and no kernel
+// of a halted iteration is launched at all.  Returns nullptr if the iteration's nodes cannot sit
+// in a conditional body (e.g. host nodes a transport adds); the caller then replays one
+// iteration per plain graph.
+template <typename F>
+static cudaGraphExec_t capture_while_graph(qudax_ctx *c, SolverScalars *S, int n, F &&body, long long *outer,
+                                           long long *per_iter) {
+    cudaGraph_t g = nullptr;
+    QX_CUDA(cudaGraphCreate(&g, 0));
+    struct Guard {
+        cudaGraph_t g;
+        ~Guard() { if (g) cudaGraphDestroy(g); }
+    } guard{g};
+    cudaGraphConditionalHandle h;
+    QX_CUDA(cudaGraphConditionalHandleCreate(&h, g, 1u, cudaGraphCondAssignDefault));
+    cudaGraph_t cg = g;
+    QX_CUDA(cudaStreamBeginCaptureToGraph(c->stream, g, nullptr, nullptr, 0, cudaStreamCaptureModeThreadLocal));
+    launch_batch_begin(S, (unsigned long long)h, n, c->stream);
+    QX_CUDA(cudaStreamEndCapture(c->stream, &cg));
+    cudaGraphNode_t first = nullptr;
+    size_t nn = 1;
+    QX_CUDA(cudaGraphGetNodes(g, &first, &nn));
+    cudaGraphNodeParams cp = {};
+    cp.type = cudaGraphNodeTypeConditional;
+    cp.conditional.handle = h;
+    cp.conditional.type = cudaGraphCondTypeWhile;
+    cp.conditional.size = 1;
+    cudaGraphNode_t cnode = nullptr;
+    QX_CUDA(cudaGraphAddNode(&cnode, g, &first, 1, &cp));
+    cudaGraph_t bg = cp.conditional.phGraph_out[0];
+    const long long l0 = c->launches;
+    c->capturing = true;
+    QX_CUDA(cudaStreamBeginCaptureToGraph(c->stream, bg, nullptr, nullptr, 0, cudaStreamCaptureModeThreadLocal));
+    try {
+        body();
+    } catch (...) {
+        cudaGraph_t tmp;
+        cudaStreamEndCapture(c->stream, &tmp);
+        c->capturing = false;
+        c->launches = l0;
+        throw;
+    }
+    cudaGraph_t bg2 = bg;
+    const cudaError_t ee = cudaStreamEndCapture(c->stream, &bg2);
+    c->capturing = false;
+    *per_iter = c->launches - l0;
+    c->launches = l0;
+    if (ee != cudaSuccess) {
+        cudaGetLastError();
+        return nullptr;
+    }
+    {  // what a conditional body may hold: kernels, memcpy / memset, empty nodes
+        size_t nb = 0;
+        QX_CUDA(cudaGraphGetNodes(bg, nullptr, &nb));
+        std::vector<cudaGraphNode_t> nodes(nb);
+        if (nb) QX_CUDA(cudaGraphGetNodes(bg, nodes.data(), &nb));
+        for (auto nd : nodes) {
+            cudaGraphNodeType ty;
+            QX_CUDA(cudaGraphNodeGetType(nd, &ty));
+            if (ty != cudaGraphNodeTypeKernel && ty != cudaGraphNodeTypeMemcpy && ty != cudaGraphNodeTypeMemset &&
+                ty != cudaGraphNodeTypeEmpty)
+                return nullptr;
+        }
+    }
+    QX_CUDA(cudaStreamBeginCaptureToGraph(c->stream, g, &cnode, nullptr, 1, cudaStreamCaptureModeThreadLocal));
+    launch_batch_end(S, c->stream);
+    QX_CUDA(cudaStreamEndCapture(c->stream, &cg));
+    cudaGraphExec_t exec = nullptr;
+    const cudaError_t ie = cudaGraphInstantiate(&exec, g, 0);
+    if (ie != cudaSuccess) {
+        cudaGetLastError();
+        return nullptr;
+    }
+    *outer = 2;
+    return exec;
+}
+
+template <typename F>
+static qudax_ctx::Graph *cached_while_graph(qudax_ctx *c, std::vector<uintptr_t> key, SolverScalars *S, int n,
+                                            F &&body) {
+    key.push_back((uintptr_t)c->gauge_epoch);
+    key.push_back((uintptr_t)c->timing);
+    for (auto &gr : c->graphs)
+        if (gr.key == key) return gr.no_while ? nullptr : &gr;
+    if (c->graphs.size() >= kMaxGraphs) {
+        auto &old = c->graphs.front();
+        if (old.exec) cudaGraphExecDestroy(old.exec);
+        release_graph_timing(c, old.trecs);
+        c->graphs.erase(c->graphs.begin());
+    }
+    qudax_ctx::Graph gr;
+    gr.key = std::move(key);
+    gr.exec = capture_while_graph(c, S, n, body, &gr.launches, &gr.per_iter);
+    gr.no_while = (gr.exec == nullptr);
+    c->graphs.push_back(std::move(gr));
+    return c->graphs.back().no_while ? nullptr : &c->graphs.back();
+}
 
 // the Schur form matpc_op applies during one solve (restored on every exit path)
 struct SchurForm {
@@ -283,7 +377,7 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     // recurrences and Algorithm R's update rule run in the reduction tails)
     SolverScalars *S = scalars(c);
     SolverScalars *hS = c->h_scal;  // pinned staging (written only after a synchronisation)
-    const int poll = sp->poll_every > 0 ? sp->poll_every : 4;
+    const int poll = sp->poll_every > 0 ? sp->poll_every : 16;
     QX_CHECK(poll <= kHistRing, QUDAX_ERR_ARG, "poll_every must be <= " + std::to_string(kHistRing));
     {
         const cd rn = cdot_of(c, Ps, r0, rs);
@@ -300,7 +394,7 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
         hS->decide = 1;
         QX_CUDA(cudaMemcpyAsync(S, hS, sizeof(*hS), cudaMemcpyHostToDevice, c->stream));
     }
-    int k = 0, updates = 0, restarts = 0;
+    int k = 0, updates = 0, restarts = 0, polls = 0, dev_batches = 0;
     bool converged = (bnorm == 0.0);
     const double V_h_all = (double)g.Vh * g.nranks;
     double flops = 0;
@@ -309,8 +403,7 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     const double matpc_flops = mm.flops * V_h_all;
     const double blas_flops_iter = 960.0 * V_h_all;  // reading Q16 (fused BLAS per iteration)
 
-    // one BiCGstab iteration, fully stream-ordered; its scalars stay on the device and every
-    // kernel is gated on S->halt (HaltGate), so the tail of a batch after an update request is void
+    // one BiCGstab iteration, fully stream-ordered; its scalars stay on the device
     auto enqueue_iteration = [&] {
         {
             void *f[3] = {rs, p, v};
@@ -332,50 +425,53 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
             blas_op_dev(c, OP_FINAL, Ps, f, co, S, COEF_RHO);          // x += a p + w s; r = s - w t; rho', beta; decide
         }
     };
-    auto enqueue_batch = [&](int n) {
-        HaltGate gate(c, &S->halt);
-        for (int j = 0; j < n; ++j) {
-            c->cap_iter = j;
-            enqueue_iteration();
-        }
-        c->cap_iter = 0;
-    };
-    // Replay batches of `poll` iterations as one CUDA graph (no per-kernel launch latency, no
-    // host synchronisation inside a batch), cached across solves.  Not with the host transport
-    // (its hooks run on the host and synchronise), which polls after every iteration.
+    // Batches of up to `poll` iterations run as one cached batch graph (capture_while_graph): the
+    // device loops over iterations and the host reads the scalars once per batch.  One iteration
+    // per host poll instead: the host transport (its hooks synchronise), eager mode, kernel
+    // timing (its event nodes cannot sit in a conditional body), and iterations a WHILE node
+    // cannot hold — those replay one iteration as a plain cached graph (or run eagerly).
     const bool host_comm = (c->comm == QUDAX_COMM_HOST);
-#ifndef QX_EAGER_TIMING
-#define QX_EAGER_TIMING 0
-#endif
-    const bool use_graph = !host_comm && !(c->flags & QUDAX_FLAG_NO_GRAPHS) && !(QX_EAGER_TIMING && c->timing);
-    const int batch = host_comm ? 1 : poll;
+    const bool use_graph = !host_comm && !(c->flags & QUDAX_FLAG_NO_GRAPHS);
     bool first = true;
 
     while (!converged && k < sp->maxiter) {
         const std::vector<qudax_ctx::TimingRec> *grecs = nullptr;
+        qudax_ctx::Graph *while_graph = nullptr;
         if (!use_graph || first) {
-            // eager (the first batch runs eagerly: it allocates the lazily-created buffers)
-            enqueue_batch(first ? 1 : batch);
+            // eager (the first iteration runs eagerly: it allocates the lazily-created buffers)
+            enqueue_iteration();
             first = false;
         } else {
-            const std::vector<uintptr_t> key = {1, (uintptr_t)Pd, (uintptr_t)Ps, (uintptr_t)batch, (uintptr_t)rs,
+            const std::vector<uintptr_t> key = {1, (uintptr_t)Pd, (uintptr_t)Ps, (uintptr_t)poll, (uintptr_t)rs,
                                                 (uintptr_t)xs, (uintptr_t)p, (uintptr_t)v, (uintptr_t)t,
                                                 (uintptr_t)r0, (uintptr_t)S, (uintptr_t)c->matpc_sym};
-            auto *gr = cached_graph(c, key, [&] { enqueue_batch(batch); });
-            if (gr) {
-                QX_CUDA(cudaGraphLaunch(gr->exec, c->stream));
-                c->launches += gr->launches;
-                grecs = &gr->trecs;
+            qudax_ctx::Graph *wg = c->timing ? nullptr : cached_while_graph(c, key, S, poll, enqueue_iteration);
+            if (wg) {
+                QX_CUDA(cudaGraphLaunch(wg->exec, c->stream));
+                c->launches += wg->launches;  // (+ per_iter x the iterations that ran, below)
             } else {
-                enqueue_batch(batch);
+                std::vector<uintptr_t> key1 = key;
+                key1[0] = 3;  // one iteration, plain graph
+                auto *gr = cached_graph(c, key1, enqueue_iteration);
+                if (gr) {
+                    QX_CUDA(cudaGraphLaunch(gr->exec, c->stream));
+                    c->launches += gr->launches;
+                    grecs = &gr->trecs;
+                } else {
+                    enqueue_iteration();
+                }
             }
+            while_graph = wg;
         }
         QX_CUDA(cudaMemcpyAsync(hS, S, sizeof(*hS), cudaMemcpyDeviceToHost, c->stream));
         QX_CUDA(cudaStreamSynchronize(c->stream));
         check_device_error(c);
+        ++polls;
+        if (while_graph) ++dev_batches;
         const SolverScalars &hs = *hS;
-        const int ran = hs.k - k;  // iterations of this batch that ran (the rest were halted)
+        const int ran = hs.k - k;  // iterations of this batch that ran
         if (grecs) harvest_graph_timing(c, *grecs, ran);
+        if (while_graph) c->launches += while_graph->per_iter * ran;
         for (int j = 0; j < ran; ++j) {
             const int kk = k + j + 1;  // 1-based iteration number
             const double rn = hs.hist[(kk - 1) % kHistRing];
@@ -438,6 +534,8 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
     st->iters = k;
     st->reliable_updates = updates;
     st->restarts = restarts;
+    st->host_polls = polls;
+    st->device_batches = dev_batches;
     if (k == 0) st->true_res_schur = bnorm > 0 ? 1.0 : 0.0;
 
     finish_solution(c, Pd, x_dev, b_e, b_o, x_e, x_o, t_e, t_o, sp->use_schur, st);

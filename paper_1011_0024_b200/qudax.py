@@ -70,7 +70,8 @@ class SolveParam(ctypes.Structure):
 class SolveStats(ctypes.Structure):
     _fields_ = [("iters", ctypes.c_int), ("reliable_updates", ctypes.c_int), ("true_res", ctypes.c_double),
                 ("true_res_schur", ctypes.c_double), ("secs", ctypes.c_double), ("flops", ctypes.c_double),
-                ("gflops", ctypes.c_double), ("restarts", ctypes.c_int)]
+                ("gflops", ctypes.c_double), ("restarts", ctypes.c_int),
+                ("host_polls", ctypes.c_int), ("device_batches", ctypes.c_int)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}

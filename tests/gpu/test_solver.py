@@ -250,10 +250,12 @@ def test_batched_equals_independent_at_config3_size(torch_cuda):
 
 def test_poll_every_and_eager_are_bitwise_identical(torch_cuda, system):
     """Algorithm R's update rule runs on the device after every iteration; the host reads the
-    scalars once per batch of poll_every iterations (one CUDA-graph replay), and an iteration that
-    asks for a reliable update voids the rest of its batch.  The iterates must therefore not
-    depend on the batch size or on graph replay: bitwise equal x, the same iteration count,
-    updates and residual history for poll_every 1 / 3 / 4 / 16 and with graphs disabled."""
+    scalars once per batch of up to poll_every iterations (one replay of a graph whose WHILE node
+    loops over the iteration on the device), and an iteration that asks for a reliable update
+    ends its batch.  The iterates must therefore not depend on the batch size or on graph replay:
+    bitwise equal x, the same iteration count, updates and residual history for poll_every
+    1 / 3 / 4 / 16 and with graphs disabled — and the batches must really run on the device
+    (device_batches, host_polls)."""
     U, wc = system
     b = qgen.point_source(DIMS, 0, 1)
     runs = []
@@ -264,6 +266,11 @@ def test_poll_every_and_eager_are_bitwise_identical(torch_cuda, system):
         x, st = ctx.solve(b, tol=1e-12, delta=1e-2, maxiter=400, prec=8, prec_sloppy=4, history=h, poll_every=poll)
         runs.append((x, st, h))
         ctx.close()
+        if flags & qudax.FLAG_NO_GRAPHS:
+            assert st["device_batches"] == 0 and st["host_polls"] == st["iters"], st
+        elif poll > 1:
+            assert st["device_batches"] >= 1, st
+            assert st["host_polls"] <= st["iters"] // poll + st["reliable_updates"] + 3, st
     x0, st0, h0 = runs[0]
     assert st0["reliable_updates"] >= 2
     for x, st, h in runs[1:]:

@@ -28,7 +28,7 @@ def test_library_exports_every_header_symbol():
 
 
 def test_abi_version_and_status_strings():
-    assert qudax.lib().qudax_abi_version() == 4
+    assert qudax.lib().qudax_abi_version() == 5
     assert qudax.status_string(0) == "ok"
     assert "unsupported" in qudax.status_string(5)
 
