@@ -47,20 +47,29 @@ __device__ __forceinline__ Cx<float> operator-(Cx<float> a, Cx<float> b) {
     return cf(__ffma2_rn(f2(b), bc(-1.f), f2(a)));
 }
 __device__ __forceinline__ Cx<float> operator*(float s, Cx<float> a) { return cf(__fmul2_rn(bc(s), f2(a))); }
-// i a as a pair: (-a.i, a.r)
-__device__ __forceinline__ float2 times_i2(Cx<float> a) { return __fmul2_rn(make_float2(a.i, a.r), make_float2(-1.f, 1.f)); }
+// i a = (-a.i, a.r) and -i a = (a.i, -a.r) as FFMA2 operands: written as the FIRST operand with
+// the scalar in the second, ptxas folds the pair swap and the one-lane negation into operand
+// modifiers and the scalar into a broadcast — one FFMA2 per complex multiply-add term, exact
+// (the sign change) and with no constant.  (The former i a = swap(a) * (-1, 1) needed that
+// constant pair in registers, which ptxas rematerialised with two moves before most uses: +10 %
+// instructions in the clover-inverse kernel, profiles/r02s_summary.md.)
+__device__ __forceinline__ float2 i_pair(Cx<float> a) { return make_float2(-a.i, a.r); }
+__device__ __forceinline__ float2 mi_pair(Cx<float> a) { return make_float2(a.i, -a.r); }
+// acc + s * (i a), acc + s * (-i a)
+__device__ __forceinline__ float2 fma_i(float2 acc, float s, Cx<float> a) { return __ffma2_rn(i_pair(a), bc(s), acc); }
+__device__ __forceinline__ float2 fma_mi(float2 acc, float s, Cx<float> a) { return __ffma2_rn(mi_pair(a), bc(s), acc); }
 __device__ __forceinline__ Cx<float> operator*(Cx<float> a, Cx<float> b) {
-    return cf(__ffma2_rn(bc(a.i), times_i2(b), __fmul2_rn(bc(a.r), f2(b))));
+    return cf(fma_i(__fmul2_rn(bc(a.r), f2(b)), a.i, b));
 }
 __device__ __forceinline__ Cx<float> conj_mul(Cx<float> a, Cx<float> b) {
-    return cf(__ffma2_rn(bc(-a.i), times_i2(b), __fmul2_rn(bc(a.r), f2(b))));
+    return cf(fma_mi(__fmul2_rn(bc(a.r), f2(b)), a.i, b));
 }
 
 // p + S i q (S = +-1): one FFMA2 in fp32 (pair swap as operand modifier)
 template <int S, typename R>
 __device__ __forceinline__ Cx<R> add_i(Cx<R> p, Cx<R> q) {
     if constexpr (sizeof(R) == 4) {
-        return cf(__ffma2_rn(make_float2(q.i, q.r), make_float2((float)-S, (float)S), f2(p)));
+        return cf(__fadd2_rn(f2(p), S > 0 ? i_pair(q) : mi_pair(q)));  // swap + one-lane negation: modifiers
     } else {
         return S > 0 ? Cx<R>{p.r - q.i, p.i + q.r} : Cx<R>{p.r + q.i, p.i - q.r};
     }
@@ -489,16 +498,15 @@ struct LinkIO {
 #endif
 #if QX_XREC
             if constexpr (sizeof(R) == 4 && (QX_XREC >> (P == 2 ? 0 : 1) & 1)) {
-                // conj(x y - z w) = x.r conj(y) - x.i swap(y) - z.r conj(w) + z.i swap(w)
-                float2 cy[3];
-#pragma unroll
-                for (int c = 0; c < 3; ++c) cy[c] = __fmul2_rn(f2(u[1][c]), make_float2(1.f, -1.f));
+                // conj(x y - z w) = x.r conj(y) - x.i swap(y) - z.r conj(w) + z.i swap(w); the
+                // conjugations, swaps and negations are operand modifiers of the first (pair)
+                // operand, the scalars broadcasts of the second — no constant pair
                 auto cross = [&](int xa, int yb, int za, int wb) {
-                    const Cx<float> xx = u[0][xa], zz = u[0][za];
-                    float2 r = __fmul2_rn(bc(xx.r), cy[yb]);
-                    r = __ffma2_rn(bc(-xx.i), make_float2(u[1][yb].i, u[1][yb].r), r);
-                    r = __ffma2_rn(bc(-zz.r), cy[wb], r);
-                    return cf(__ffma2_rn(bc(zz.i), make_float2(u[1][wb].i, u[1][wb].r), r));
+                    const Cx<float> xx = u[0][xa], zz = u[0][za], y = u[1][yb], w = u[1][wb];
+                    float2 r = __fmul2_rn(make_float2(y.r, -y.i), bc(xx.r));
+                    r = __ffma2_rn(make_float2(-y.i, -y.r), bc(xx.i), r);
+                    r = __ffma2_rn(make_float2(-w.r, w.i), bc(zz.r), r);
+                    return cf(__ffma2_rn(make_float2(w.i, w.r), bc(zz.i), r));
                 };
                 const Cx<float> a0 = cross(1, 2, 2, 1), a1 = cross(2, 0, 0, 2), a2 = cross(0, 1, 1, 0);
                 u[2][0] = a0; u[2][1] = a1; u[2][2] = a2;

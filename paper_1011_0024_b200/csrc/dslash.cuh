@@ -31,18 +31,15 @@ namespace qx {
 
 template <typename R>
 __device__ __forceinline__ void su3_mul(const Cx<R> u[3][3], const Cx<R> v[3], Cx<R> out[3]) {
-    if constexpr (sizeof(R) == 4) {  // 1 + 6 FFMA2 per row, i v shared by the rows
-        float2 iv[3];
-#pragma unroll
-        for (int c = 0; c < 3; ++c) iv[c] = times_i2(v[c]);
+    if constexpr (sizeof(R) == 4) {  // 1 FMUL2 + 5 FFMA2 per row (fma_i: modifiers, no i v temporaries)
 #pragma unroll
         for (int a = 0; a < 3; ++a) {
             float2 acc = __fmul2_rn(bc(u[a][0].r), f2(v[0]));
-            acc = __ffma2_rn(bc(u[a][0].i), iv[0], acc);
+            acc = fma_i(acc, u[a][0].i, v[0]);
 #pragma unroll
             for (int c = 1; c < 3; ++c) {
                 acc = __ffma2_rn(bc(u[a][c].r), f2(v[c]), acc);
-                acc = __ffma2_rn(bc(u[a][c].i), iv[c], acc);
+                acc = fma_i(acc, u[a][c].i, v[c]);
             }
             out[a] = cf(acc);
         }
@@ -55,17 +52,14 @@ __device__ __forceinline__ void su3_mul(const Cx<R> u[3][3], const Cx<R> v[3], C
 template <typename R>
 __device__ __forceinline__ void su3_dag_mul(const Cx<R> u[3][3], const Cx<R> v[3], Cx<R> out[3]) {
     if constexpr (sizeof(R) == 4) {
-        float2 iv[3];
-#pragma unroll
-        for (int c = 0; c < 3; ++c) iv[c] = times_i2(v[c]);
 #pragma unroll
         for (int a = 0; a < 3; ++a) {
             float2 acc = __fmul2_rn(bc(u[0][a].r), f2(v[0]));
-            acc = __ffma2_rn(bc(-u[0][a].i), iv[0], acc);
+            acc = fma_mi(acc, u[0][a].i, v[0]);
 #pragma unroll
             for (int c = 1; c < 3; ++c) {
                 acc = __ffma2_rn(bc(u[c][a].r), f2(v[c]), acc);
-                acc = __ffma2_rn(bc(-u[c][a].i), iv[c], acc);
+                acc = fma_mi(acc, u[c][a].i, v[c]);
             }
             out[a] = cf(acc);
         }
@@ -334,12 +328,9 @@ __device__ __forceinline__ void temporal_hop(const R *hv, const Cx<R> u[3][3], R
 template <typename R>
 __device__ __forceinline__ void herm6_mul(const R *m, const Cx<R> v[6], Cx<R> out[6]) {
     if constexpr (sizeof(R) == 4) {  // out_i += L v_j and out_j += conj(L) v_i: 2 FFMA2 each
-        float2 iv[6], o[6];
+        float2 o[6];
 #pragma unroll
-        for (int i = 0; i < 6; ++i) {
-            iv[i] = times_i2(v[i]);
-            o[i] = __fmul2_rn(bc(m[i]), f2(v[i]));
-        }
+        for (int i = 0; i < 6; ++i) o[i] = __fmul2_rn(bc(m[i]), f2(v[i]));
 #pragma unroll
         for (int i = 1; i < 6; ++i)
 #pragma unroll
@@ -347,9 +338,9 @@ __device__ __forceinline__ void herm6_mul(const R *m, const Cx<R> v[6], Cx<R> ou
                 const int k = i * (i - 1) / 2 + j;
                 const float Lr = m[6 + 2 * k], Li = m[6 + 2 * k + 1];
                 o[i] = __ffma2_rn(bc(Lr), f2(v[j]), o[i]);
-                o[i] = __ffma2_rn(bc(Li), iv[j], o[i]);
+                o[i] = fma_i(o[i], Li, v[j]);
                 o[j] = __ffma2_rn(bc(Lr), f2(v[i]), o[j]);
-                o[j] = __ffma2_rn(bc(-Li), iv[i], o[j]);
+                o[j] = fma_mi(o[j], Li, v[i]);
             }
 #pragma unroll
         for (int i = 0; i < 6; ++i) out[i] = cf(o[i]);
