@@ -56,6 +56,14 @@ __global__ void k_batch_begin(SolverScalars *S, unsigned long long cond, int n) 
     S->kstop = S->k + n;
 }
 __global__ void k_batch_end(SolverScalars *S) { S->cond = 0ull; }
+// last node of the WHILE body: stop the loop after this iteration if the host must act
+// (reliable update, convergence, maxiter: S->halt) or the batch is complete.  A kernel of its
+// own so that the heavy kernels carry no conditional-handle call (ncu cannot profile kernels
+// that can set a graph condition)
+__global__ void k_batch_cond(const SolverScalars *S) {
+    cudaGraphSetConditional((cudaGraphConditionalHandle)S->cond, (S->halt || S->k >= S->kstop) ? 0u : 1u);
+}
+void launch_batch_cond(const SolverScalars *S, cudaStream_t s) { k_batch_cond<<<1, 1, 0, s>>>(S); }
 void launch_batch_begin(SolverScalars *S, unsigned long long cond, int n, cudaStream_t s) {
     k_batch_begin<<<1, 1, 0, s>>>(S, cond, n);
 }

@@ -84,9 +84,9 @@ inline int spatial_split(const Geom &g) { return g.split & 7; }
 // The iteration's update rule (Algorithm R, solver.cpp) is evaluated on the device right after
 // the |r|^2 reduction (COEF_RHO with decide != 0): the host reads the scalars once per batch of
 // up to `poll_every` iterations instead of after every iteration.  A batch is a CUDA graph whose
-// WHILE node repeats one iteration while the condition `cond` holds; the tail that evaluates
-// the rule clears it when the iteration calls for a reliable update (`halt`), converged, or
-// completes the batch (k == kstop) — so no further kernel of the batch is launched at all, and
+// WHILE node repeats one iteration while the condition `cond` holds; the iteration's last
+// kernel (k_batch_cond) clears it when the tail that evaluates the rule asked for a reliable
+// update (`halt`: also convergence and maxiter) or the batch is complete (k == kstop) — so no further kernel of the batch is launched at all, and
 // the iterates are exactly those of a host decision taken after every iteration.
 constexpr int kHistRing = 64;  // per-iteration |r| of the current batch (poll_every <= kHistRing)
 struct SolverScalars {
@@ -322,6 +322,7 @@ int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co,
 void launch_coef(SolverScalars *S, int mode, cudaStream_t s);
 void launch_batch_begin(SolverScalars *S, unsigned long long cond, int n, cudaStream_t s);
 void launch_batch_end(SolverScalars *S, cudaStream_t s);
+void launch_batch_cond(const SolverScalars *S, cudaStream_t s);
 // flags[2 mu], flags[2 mu + 1] = ++*seq for every mu in mask (NCCL halo tail mode)
 void launch_raise_flags(unsigned *flags, unsigned *seq, int mask, cudaStream_t s);
 void blas_xpy_mixed(int pd, int ps, const Geom &g, const void *x, void *y, cudaStream_t s);

@@ -57,10 +57,6 @@ __device__ __forceinline__ void apply_coef(SolverScalars *S, int mode) {
                 S->blown = blown;
                 S->halt = 1;
             }
-            // inside a batch graph: stop its WHILE node after this iteration if the host must act
-            // (reliable update, convergence, maxiter) or the batch is complete
-            if (S->cond)
-                cudaGraphSetConditional((cudaGraphConditionalHandle)S->cond, (S->halt || S->k >= S->kstop) ? 0u : 1u);
         }
     }
 }

@@ -165,10 +165,10 @@ static qudax_ctx::Graph *cached_graph(qudax_ctx *c, std::vector<uintptr_t> key, 
     return &c->graphs.back();
 }
 
-// Batch graph (solve_dev): [k_batch_begin] -> WHILE(cond) { one iteration } -> [k_batch_end].
-// The WHILE node repeats the captured iteration on the device until the reduction tail that
-// evaluates Algorithm R clears the condition (reliable update, convergence, maxiter, or the
-// batch's `n` iterations done): no host round trip and no launch inside a batch, and no kernel
+// Batch graph (solve_dev): [k_batch_begin] -> WHILE(cond) { one iteration; k_batch_cond } ->
+// [k_batch_end].  The WHILE node repeats the captured iteration on the device until k_batch_cond
+// clears the condition from what the reduction tail evaluating Algorithm R decided (reliable
+// update, convergence, maxiter) or after the batch's `n` iterations: no host round trip and no launch inside a batch, and no kernel
 // of a halted iteration is launched at all.  Returns nullptr if the iteration's nodes cannot sit
 // in a conditional body (e.g. host nodes a transport adds); the caller then replays one
 // iteration per plain graph.
@@ -203,6 +203,7 @@ static cudaGraphExec_t capture_while_graph(qudax_ctx *c, SolverScalars *S, int n
     QX_CUDA(cudaStreamBeginCaptureToGraph(c->stream, bg, nullptr, nullptr, 0, cudaStreamCaptureModeThreadLocal));
     try {
         body();
+        launch_batch_cond(S, c->stream);
     } catch (...) {
         cudaGraph_t tmp;
         cudaStreamEndCapture(c->stream, &tmp);
@@ -213,7 +214,7 @@ static cudaGraphExec_t capture_while_graph(qudax_ctx *c, SolverScalars *S, int n
     cudaGraph_t bg2 = bg;
     const cudaError_t ee = cudaStreamEndCapture(c->stream, &bg2);
     c->capturing = false;
-    *per_iter = c->launches - l0;
+    *per_iter = c->launches - l0 + 1;  // + k_batch_cond
     c->launches = l0;
     if (ee != cudaSuccess) {
         cudaGetLastError();
