@@ -454,10 +454,12 @@ __host__ __device__ constexpr bool dslash_pair() {
 #define QX_DSLASH_THREADS 128
 #endif
 // Minimum resident CTAs per SM (register cap).  Measured on B200 at 32^3x64
-// (profiles/r01_variants.log): fp32 / half need >= 6 x 128 threads in flight per SM to cover
-// HBM latency (80 regs; with the packed FP32x2 math 7 x 128 = 72 regs spilled more and lost
-// 3-8%), fp64 must not be capped (152 regs; capping spills and loses 20%).
-template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) ? 1 : 6; };
+// (profiles/r01_variants.log, profiles/r02y_*): fp32 needs >= 6 x 128 threads in flight per SM
+// to cover HBM latency (80 regs; 7 x 128 = 72 regs spills and loses up to 3 % on the xpay); half
+// runs 7 x 128 (72 regs: since the i-multiplications became operand modifiers its few spills
+// cost less than the extra warps gain, -3 % per kernel, r02y; round 1 measured 6 better); fp64
+// must not be capped (152 regs; capping spills and loses 20 %).
+template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) ? 1 : (P == 2 ? 7 : 6); };
 #ifdef QX_DSLASH_MINB
 #define QX_MINB_OF(P) QX_DSLASH_MINB
 #else
@@ -482,6 +484,60 @@ __device__ __forceinline__ void pf_spinor_l1(const void *base, long stride, long
         for (int k = 0; k < NB; ++k) pf_l1(cptr(base, (size_t)16 * (k * stride + j)));
     }
 }
+// The fused reductions' per-site partials (reading R5: the 24-term sums in the kernel's
+// arithmetic precision, accumulated over sites in fp64): (<out, w>, |out|^2) for RED_XDOT_NORM
+// (w = x), <w, out> for RED_RHAT_DOT (w = rhat0).  fp32: three packed lane-wise sums
+// A = sum o (.) w, B = sum o (.) swap(w), C = sum o (.) o (one FFMA2 each per complex value;
+// the swap is an operand modifier), combined at the end: Re = A.x + A.y, Im = B.x - B.y
+// (resp. B.y - B.x), |o|^2 = C.x + C.y.  Shared by the single- and multi-RHS kernels so that
+// a batched solve stays bitwise its independent solves.
+template <typename R>
+__device__ __forceinline__ void site_partials(const R *o, const R *w, int red_kind, double *red) {
+#ifndef QX_RED_SITE_F64
+    if constexpr (sizeof(R) == 4) {
+        float2 A = __fmul2_rn(make_float2(o[0], o[1]), make_float2(w[0], w[1]));
+        float2 B = __fmul2_rn(make_float2(o[0], o[1]), make_float2(w[1], w[0]));
+#pragma unroll
+        for (int k = 1; k < 12; ++k) {
+            A = __ffma2_rn(make_float2(o[2 * k], o[2 * k + 1]), make_float2(w[2 * k], w[2 * k + 1]), A);
+            B = __ffma2_rn(make_float2(o[2 * k], o[2 * k + 1]), make_float2(w[2 * k + 1], w[2 * k]), B);
+        }
+        if (red_kind == RED_XDOT_NORM) {
+            float2 C = __fmul2_rn(make_float2(o[0], o[1]), make_float2(o[0], o[1]));
+#pragma unroll
+            for (int k = 1; k < 12; ++k)
+                C = __ffma2_rn(make_float2(o[2 * k], o[2 * k + 1]), make_float2(o[2 * k], o[2 * k + 1]), C);
+            red[0] += (double)(A.x + A.y);
+            red[1] += (double)(B.x - B.y);
+            red[2] += (double)(C.x + C.y);
+        } else {
+            red[0] += (double)(A.x + A.y);
+            red[1] += (double)(B.y - B.x);
+        }
+        return;
+    }
+    using RA = R;
+#else
+    using RA = double;
+#endif
+    RA s0 = 0, s1 = 0, s2 = 0;
+#pragma unroll
+    for (int k = 0; k < 12; ++k) {
+        const RA orr = o[2 * k], oi = o[2 * k + 1], wr = w[2 * k], wi = w[2 * k + 1];
+        if (red_kind == RED_XDOT_NORM) {  // (<out, x>, |out|^2)
+            s0 += orr * wr + oi * wi;
+            s1 += orr * wi - oi * wr;
+            s2 += orr * orr + oi * oi;
+        } else {                          // <rhat, out>
+            s0 += wr * orr + wi * oi;
+            s1 += wr * oi - wi * orr;
+        }
+    }
+    red[0] += (double)s0;
+    red[1] += (double)s1;
+    red[2] += (double)s2;
+}
+
 // one output site; red[] receives this site's contribution to the optional fused reduction
 // INMODE: load mode of the neighbour spinors (0 read-only path; 2 L2-coherent, for inputs
 // written by other CTAs earlier in the same launch — the fused Mhat kernel)
@@ -787,27 +843,7 @@ __device__ __forceinline__ void dslash_site(const DslashArgs &a, const void *fin
     // (multi-RHS launch: this CTA's right-hand side, recomputed here rather than kept live)
     const void *rh = a.nrhs > 1 ? a.rhat_m[blockIdx.x % a.nrhs] : a.rhat;
     SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx : rh, a.stride, i, w);
-#ifdef QX_RED_SITE_F64
-    using RA = double;
-#else
-    using RA = R;  // the site's 24-term partial in the arithmetic precision, sites summed in fp64
-#endif
-    RA s0 = 0, s1 = 0, s2 = 0;
-#pragma unroll
-    for (int k = 0; k < 12; ++k) {
-        const RA orr = o[2 * k], oi = o[2 * k + 1], wr = w[2 * k], wi = w[2 * k + 1];
-        if (a.red_kind == RED_XDOT_NORM) {  // (<out, x>, |out|^2)
-            s0 += orr * wr + oi * wi;
-            s1 += orr * wi - oi * wr;
-            s2 += orr * orr + oi * oi;
-        } else {                             // <rhat, out>
-            s0 += wr * orr + wi * oi;
-            s1 += wr * oi - wi * orr;
-        }
-    }
-    red[0] += (double)s0;
-    red[1] += (double)s1;
-    red[2] += (double)s2;
+    site_partials<R>(o, w, a.red_kind, red);
 }
 
 // Kernel-initiated halo (QUDAX_HALO_P2P): one thread per CTA acquires the two flags the

@@ -283,27 +283,7 @@ __device__ __forceinline__ void dslash_site_mr(const DslashArgs &a, int tid, int
         SpinorIO<P>::store_requant(fout[r], a.stride, i, o);
         R w[24];
         SpinorIO<P>::load(a.red_kind == RED_XDOT_NORM ? fx[r] : frh[r], a.stride, i, w);
-#ifdef QX_RED_SITE_F64
-        using RA = double;
-#else
-        using RA = R;
-#endif
-        RA s0 = 0, s1 = 0, s2 = 0;
-#pragma unroll
-        for (int k = 0; k < 12; ++k) {
-            const RA orr = o[2 * k], oi = o[2 * k + 1], wr = w[2 * k], wi = w[2 * k + 1];
-            if (a.red_kind == RED_XDOT_NORM) {
-                s0 += orr * wr + oi * wi;
-                s1 += orr * wi - oi * wr;
-                s2 += orr * orr + oi * oi;
-            } else {
-                s0 += wr * orr + wi * oi;
-                s1 += wr * oi - wi * orr;
-            }
-        }
-        red[r][0] += (double)s0;
-        red[r][1] += (double)s1;
-        red[r][2] += (double)s2;
+        site_partials<R>(o, w, a.red_kind, red[r]);
     }
 }
 
