@@ -31,6 +31,12 @@ import time
 
 ROOT = os.path.dirname(os.path.abspath(__file__))
 sys.path.insert(0, ROOT)
+# NCCL's graph-mixing support adds an external event-wait node to every NCCL operation captured
+# in a graph, which a conditional (WHILE) graph body cannot hold: with it, a partitioned solve
+# falls back to one host poll per iteration (the library prints why).  The library never runs
+# graph-captured and eager NCCL work of one communicator concurrently, so the bench (the NCCL
+# user of this process) switches it off before NCCL initialises (profiles/r02ab_*).
+os.environ.setdefault("NCCL_GRAPH_MIXING_SUPPORT", "0")
 
 METRIC = "Dslash GFLOPS & HBM GB/s per B200 at 1/2/4/8 GPUs; mixed-prec solve time"
 KAPPA, CSW, EPS = 0.124, 1.0, 0.1

@@ -740,16 +740,18 @@ void matpc_sym_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger,
     blas_op(c, OP_XPAY, prec, f, &a, nullptr);
 }
 
-void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red) {
+void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red, int order) {
     if (c->matpc_sym) {
         matpc_sym_op(c, out, in, prec, dagger, red);
         return;
     }
     void *t = tmp_odd(c, prec);
-    dslash_op(c, t, in, nullptr, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, nullptr);
-    // the second kernel walks the lattice top-down: the timeslices the first kernel touched
-    // last (their links, T^{-1} D in and the dirty tmp lines) are still in the 126 MB L2
-    dslash_op(c, out, t, in, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, red, QX_MATPC_REVERSE);
+    // the two kernels walk the lattice in opposite directions: the second starts on the
+    // timeslices the first touched last (their links, T^{-1} D in and the dirty tmp lines are
+    // still in the 126 MB L2)
+    dslash_op(c, t, in, nullptr, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, nullptr, order ? 1 : 0);
+    dslash_op(c, out, t, in, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, red,
+              order ? 0 : QX_MATPC_REVERSE);
 }
 
 // Multi-RHS Dslash (SURVEY NEXT row 2, P:748-753 / P:1092-1094: many right-hand sides per
@@ -875,7 +877,7 @@ void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, cons
 }
 
 void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger,
-                    const RedReq *reds) {
+                    const RedReq *reds, int order) {
     QX_CHECK(n >= 1 && n <= kMaxRhs, QUDAX_ERR_ARG, "nrhs must be 1.." + std::to_string(kMaxRhs));
     void *t[kMaxRhs];
     for (int k = 0; k < n; ++k) {
@@ -884,8 +886,10 @@ void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n
         t[k] = slot;
     }
     QX_CHECK(!c->matpc_sym, QUDAX_ERR_UNSUPPORTED, "multi-RHS Mhat: asymmetric Schur form only");
-    dslash_multi_op(c, t, in, nullptr, n, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, 0, nullptr);
-    dslash_multi_op(c, out, t, in, n, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa, 1, reds);
+    // (the same kernel directions as matpc_op, so a batched solve stays bitwise its single ones)
+    dslash_multi_op(c, t, in, nullptr, n, prec, 1, dagger, QUDAX_CLOVER_INV, 0.0, order ? 1 : 0, nullptr);
+    dslash_multi_op(c, out, t, in, n, prec, 0, dagger, QUDAX_CLOVER_XPAY, -c->kappa * c->kappa,
+                    order ? 0 : QX_MATPC_REVERSE, reds);
 }
 
 void clover_apply_op(qudax_ctx *c, void *out, const void *in, int prec, int parity, bool inverse) {

@@ -116,11 +116,12 @@ __global__ void k_p_update(long Vh, long stride, const void *r, void *p, const v
 
 // y <- y + c x   (c complex)
 template <int P>
-__global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y) {
+__global__ void k_caxpy(long Vh, long stride, CoefArg c_, const void *x, void *y, int rev) {
     using R = typename Prec<P>::R;
     const double2 c = coef_get(c_);
     const Cx<R> a = cx((R)c.x, (R)c.y);
-    QX_GRID_LOOP(i) {
+    QX_GRID_LOOP(j) {
+        const long i = rev ? Vh - 1 - j : j;  // (top-down: start where the previous kernel ended)
         R xx[24], yy[24];
         SpinorIO<P>::load(x, stride, i, xx);
         SpinorIO<P>::load(y, stride, i, yy);
@@ -347,7 +348,10 @@ int blas_run(int op, int prec, const Geom &g, void *const *f, const CoefArg *co,
             QX_PREC_SWITCH(prec, QX_LAUNCH(k_p_update<P>, Vh, st, f[0], f[1], f[2], co[0], co[1]));
             break;
         case OP_CAXPY:  // f1 += c f0
-            QX_PREC_SWITCH(prec, QX_LAUNCH(k_caxpy<P>, Vh, st, co[0], f[0], f[1]));
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_caxpy<P>, Vh, st, co[0], f[0], f[1], 0));
+            break;
+        case OP_CAXPY_REV:
+            QX_PREC_SWITCH(prec, QX_LAUNCH(k_caxpy<P>, Vh, st, co[0], f[0], f[1], 1));
             break;
         case OP_XPAY:  // f2 = f0 + a f1
             QX_PREC_SWITCH(prec, QX_LAUNCH(k_xpay<P>, Vh, st, f[0], co[0].v.x, f[1], f[2]));

@@ -176,12 +176,15 @@ struct RedReq {
 };
 void dslash_op(qudax_ctx *c, void *out, const void *in, const void *x, int prec, int p, int dagger, int kind,
                double a, const RedReq *red = nullptr, int reverse = 0);
-void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr);
+// order 0: first kernel bottom-up, second top-down; order 1: the reverse (solver.cpp: each kernel
+// starts where the previous one ended, so the first fields it reads are still in L2)
+void matpc_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr,
+              int order = 0);
 void matpc_sym_op(qudax_ctx *c, void *out, const void *in, int prec, int dagger, const RedReq *red = nullptr);
 void dslash_multi_op(qudax_ctx *c, void *const *out, const void *const *in, const void *const *x, int n, int prec,
                      int p, int dagger, int kind, double a, int reverse, const RedReq *reds = nullptr);
 void matpc_multi_op(qudax_ctx *c, void *const *out, const void *const *in, int n, int prec, int dagger,
-                    const RedReq *reds = nullptr);
+                    const RedReq *reds = nullptr, int order = 0);
 void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_dev, int n, const qudax_solve_param *p,
                      qudax_solve_stats *st);
 int dslash_threads();

@@ -306,7 +306,8 @@ void launch_clover_apply(int prec, const Geom &g, const void *cl, const void *in
 // BLAS / reductions (blas.cu).  ops: 0 p_update, 1 caxpy, 2 xpay, 3 cdot, 4 norm2, 5 tdot,
 // 6 bicgstab final update, 7 r = b - r with |r|^2.  Returns the number of reduced doubles
 // written to `out` (device).
-enum BlasOp { OP_P_UPDATE = 0, OP_CAXPY, OP_XPAY, OP_CDOT, OP_NORM2, OP_TDOT, OP_FINAL, OP_BMR_NORM };
+// OP_CAXPY_REV: OP_CAXPY walking the sites top-down (the solver's L2-aware kernel order)
+enum BlasOp { OP_P_UPDATE = 0, OP_CAXPY, OP_XPAY, OP_CDOT, OP_NORM2, OP_TDOT, OP_FINAL, OP_BMR_NORM, OP_CAXPY_REV };
 // a BLAS coefficient: the value v, or (d != nullptr) a device scalar read by the kernel
 struct CoefArg {
     double2 v;

@@ -165,6 +165,16 @@ static qudax_ctx::Graph *cached_graph(qudax_ctx *c, std::vector<uintptr_t> key, 
     return &c->graphs.back();
 }
 
+// Kernel directions of a BiCGstab iteration (QX_SOLVER_ORDER 1): every kernel starts at the end
+// of the lattice where the previous one finished, so the first part of the field it reads from
+// the previous kernel (p, tmp, v, s, tmp, t) is still in the 126 MB L2 — p update (up), first
+// Mhat's clover-inverse kernel (down) and xpay (up), s = r - alpha v (down), second Mhat's
+// kernels (up, down), final update (up): six of the seven transitions hot instead of four.
+#ifndef QX_SOLVER_ORDER
+#define QX_SOLVER_ORDER 1
+#endif
+constexpr int kCaxpyOp = QX_SOLVER_ORDER ? OP_CAXPY_REV : OP_CAXPY;
+
 // Batch graph (solve_dev): [k_batch_begin] -> WHILE(cond) { one iteration; k_batch_cond } ->
 // [k_batch_end].  The WHILE node repeats the captured iteration on the device until k_batch_cond
 // clears the condition from what the reduction tail evaluating Algorithm R decided (reliable
@@ -217,6 +227,8 @@ static cudaGraphExec_t capture_while_graph(qudax_ctx *c, SolverScalars *S, int n
     *per_iter = c->launches - l0 + 1;  // + k_batch_cond
     c->launches = l0;
     if (ee != cudaSuccess) {
+        std::fprintf(stderr, "qudax: capture of the batch iteration into a WHILE body failed (%s); one iteration per host poll\n",
+                     cudaGetErrorString(ee));
         cudaGetLastError();
         return nullptr;
     }
@@ -229,8 +241,11 @@ static cudaGraphExec_t capture_while_graph(qudax_ctx *c, SolverScalars *S, int n
             cudaGraphNodeType ty;
             QX_CUDA(cudaGraphNodeGetType(nd, &ty));
             if (ty != cudaGraphNodeTypeKernel && ty != cudaGraphNodeTypeMemcpy && ty != cudaGraphNodeTypeMemset &&
-                ty != cudaGraphNodeTypeEmpty)
+                ty != cudaGraphNodeTypeEmpty) {
+                std::fprintf(stderr, "qudax: the batch iteration holds a graph node of type %d (of %zu nodes) a WHILE "
+                             "body cannot; one iteration per host poll\n", (int)ty, nb);
                 return nullptr;
+            }
         }
     }
     QX_CUDA(cudaStreamBeginCaptureToGraph(c->stream, g, &cnode, nullptr, 1, cudaStreamCaptureModeThreadLocal));
@@ -239,6 +254,8 @@ static cudaGraphExec_t capture_while_graph(qudax_ctx *c, SolverScalars *S, int n
     cudaGraphExec_t exec = nullptr;
     const cudaError_t ie = cudaGraphInstantiate(&exec, g, 0);
     if (ie != cudaSuccess) {
+        std::fprintf(stderr, "qudax: instantiating the WHILE batch graph failed (%s); one iteration per host poll\n",
+                     cudaGetErrorString(ie));
         cudaGetLastError();
         return nullptr;
     }
@@ -412,11 +429,11 @@ void solve_dev(qudax_ctx *c, double *x_dev, const double *b_dev, const qudax_sol
             blas_op_dev(c, OP_P_UPDATE, Ps, f, co, S, COEF_NONE);      // p = r + beta (p - omega v)
         }
         RedReq red_rv{RED_RHAT_DOT, r0, nullptr, S, COEF_ALPHA};
-        matpc_op(c, v, p, Ps, 0, &red_rv);                            // v = Mhat p; alpha = rho'/<rhat0,v>
+        matpc_op(c, v, p, Ps, 0, &red_rv, QX_SOLVER_ORDER);           // v = Mhat p; alpha = rho'/<rhat0,v>
         {
             void *f[2] = {v, rs};
             CoefArg co[1] = {{{0, 0}, &S->malpha}};
-            blas_op_dev(c, OP_CAXPY, Ps, f, co, S, COEF_NONE);         // s = r - alpha v
+            blas_op_dev(c, kCaxpyOp, Ps, f, co, S, COEF_NONE);         // s = r - alpha v
         }
         RedReq red_ts{RED_XDOT_NORM, nullptr, nullptr, S, COEF_OMEGA};
         matpc_op(c, t, rs, Ps, 0, &red_ts);                            // t = Mhat s; omega = <t,s>/|t|^2
@@ -629,12 +646,12 @@ void solve_multi_dev(qudax_ctx *c, double *const *x_dev, const double *const *b_
             red_ts[na] = RedReq{RED_XDOT_NORM, nullptr, nullptr, y.S, COEF_OMEGA};
             ++na;
         }
-        matpc_multi_op(c, vv, pp, na, Ps, 0, red_rv);  // v = Mhat p; alpha = rho'/<rhat0, v>
+        matpc_multi_op(c, vv, pp, na, Ps, 0, red_rv, QX_SOLVER_ORDER);  // v = Mhat p; alpha = rho'/<rhat0, v>
         for (int j = 0; j < n; ++j) {
             if (!(mask >> j & 1)) continue;
             void *f[2] = {sys[j].v, sys[j].rs};
             CoefArg co[1] = {{{0, 0}, &sys[j].S->malpha}};
-            blas_op_dev(c, OP_CAXPY, Ps, f, co, sys[j].S, COEF_NONE);  // s = r - alpha v
+            blas_op_dev(c, kCaxpyOp, Ps, f, co, sys[j].S, COEF_NONE);  // s = r - alpha v
         }
         matpc_multi_op(c, tt, ss, na, Ps, 0, red_ts);  // t = Mhat s; omega = <t,s>/|t|^2
         for (int j = 0; j < n; ++j) {
