@@ -328,3 +328,56 @@ def test_binding_rejects_bad_buffers(torch_cuda, system):
     with pytest.raises(ValueError):
         ctx.matpc(ctx.new_field(2), ctx.new_field(2), 4)  # half-sized buffers for an fp32 operator
     ctx.close()
+
+
+_WHILE_NCCL_CHILD = r"""
+import hashlib, json, sys
+import numpy as np
+sys.path.insert(0, sys.argv[1])
+import qgen
+from paper_1011_0024_b200 import qudax
+dims = (8, 8, 8, 16)
+U = qgen.gauge(dims, 1003, eps=0.1)
+b = qgen.point_source(dims, 1, 2)
+out = {}
+for comm in (qudax.COMM_NONE, qudax.COMM_NCCL):
+    for ov in ((False,) if comm == qudax.COMM_NONE else (False, True)):
+        ctx = qudax.Context(dims, comm=comm, overlap=ov, nccl_id=qudax.nccl_unique_id() if comm else None)
+        ctx.gauge_load(U, 0.124, 1.0, prec=8, recon=18, prec_sloppy=4, recon_sloppy=12)
+        for _ in range(2):  # the second solve replays the cached batch graph
+            x, st = ctx.solve(b, tol=1e-11, delta=1e-2, maxiter=400, prec=8, prec_sloppy=4)
+        out[f"{comm}-{int(ov)}"] = {"x": hashlib.sha256(x.tobytes()).hexdigest(), "iters": st["iters"],
+                                     "device_batches": st["device_batches"], "host_polls": st["host_polls"],
+                                     "true_res": st["true_res"]}
+        ctx.close()
+print(json.dumps(out))
+"""
+
+
+def test_nccl_loopback_iterations_in_while_node(torch_cuda, tmp_path):
+    """The N > 1 solver path with the device-side batch loop: with NCCL's graph-mixing support off
+    (it adds event-wait nodes a conditional graph body cannot hold; bench.py switches it off),
+    the NCCL-loopback iteration — halo send/recv and the allreduce of the fused sums, with and
+    without the overlapped tail launch — runs inside the WHILE node (device_batches > 0, far
+    fewer host polls than iterations); without overlap (one whole-lattice kernel, the unsplit
+    reduction grouping) it is bitwise the unsplit solve, with overlap within the tolerance.  A
+    child process, so the NCCL environment is set before NCCL initialises."""
+    import json
+    import os
+    import subprocess
+    import sys
+    root = os.path.dirname(os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+    env = dict(os.environ, NCCL_GRAPH_MIXING_SUPPORT="0")
+    r = subprocess.run([sys.executable, "-c", _WHILE_NCCL_CHILD, root], env=env, capture_output=True, text=True,
+                       timeout=600)
+    assert r.returncode == 0, r.stderr[-2000:]
+    out = json.loads(r.stdout.strip().splitlines()[-1])
+    ref = out["0-0"]
+    assert ref["device_batches"] > 0
+    for key in ("1-0", "1-1"):
+        st = out[key]
+        assert st["device_batches"] > 0, (key, st, r.stderr[-1000:])
+        assert st["host_polls"] < st["iters"], (key, st)
+        assert st["true_res"] <= 1e-11 * (1 + 1e-3), (key, st)
+    st = out["1-0"]
+    assert st["iters"] == ref["iters"] and st["x"] == ref["x"] and st["true_res"] == ref["true_res"], (st, ref)
