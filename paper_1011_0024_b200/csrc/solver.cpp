@@ -278,7 +278,22 @@ static qudax_ctx::Graph *cached_while_graph(qudax_ctx *c, std::vector<uintptr_t>
     }
     qudax_ctx::Graph gr;
     gr.key = std::move(key);
-    gr.exec = capture_while_graph(c, S, n, body, &gr.launches, &gr.per_iter);
+    try {
+        gr.exec = capture_while_graph(c, S, n, body, &gr.launches, &gr.per_iter);
+    } catch (const Error &e) {
+        // a runtime without conditional nodes, or a capture it refuses: one iteration per poll
+        if (e.status != QUDAX_ERR_CUDA && e.status != QUDAX_ERR_NCCL) throw;
+        cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
+        if (cudaStreamIsCapturing(c->stream, &cs) == cudaSuccess && cs != cudaStreamCaptureStatusNone) {
+            cudaGraph_t tmp = nullptr;
+            cudaStreamEndCapture(c->stream, &tmp);
+            if (tmp) cudaGraphDestroy(tmp);
+        }
+        c->capturing = false;
+        cudaGetLastError();
+        std::fprintf(stderr, "qudax: WHILE batch graph unavailable (%s); one iteration per host poll\n", e.what());
+        gr.exec = nullptr;
+    }
     gr.no_while = (gr.exec == nullptr);
     c->graphs.push_back(std::move(gr));
     return c->graphs.back().no_while ? nullptr : &c->graphs.back();
