@@ -465,6 +465,21 @@ template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) 
 #else
 #define QX_MINB_OF(P) DslashMinBlocks<P>::value
 #endif
+// eight-parameter links (sincos / sqrt reconstruction): half recon-8 needs the registers of
+// 6 CTAs per SM (at 7 it spills 156 B: 125.2 vs 121.4 us clover-inverse, r02aj); fp32 recon-8
+// stays at 6 (5 CTAs: 143.9 vs 141.7 us)
+#ifndef QX_R8_MINB_F32
+#define QX_R8_MINB_F32 6
+#endif
+#ifndef QX_R8_MINB_F16
+#define QX_R8_MINB_F16 6
+#endif
+#ifdef QX_DSLASH_MINB
+#define QX_MINB_OF2(P, RECON) QX_DSLASH_MINB
+#else
+#define QX_MINB_OF2(P, RECON) \
+    ((RECON) == 8 && (P) == 4 ? QX_R8_MINB_F32 : ((RECON) == 8 && (P) == 2 ? QX_R8_MINB_F16 : DslashMinBlocks<P>::value))
+#endif
 // L1 prefetch (QX_RED_PF: the fused reduction's second operand, see dslash_site)
 __device__ __forceinline__ void pf_l1(const void *p) { asm volatile("prefetch.global.L1 [%0];" ::"l"(p)); }
 #ifndef QX_RED_PF
@@ -905,7 +920,7 @@ static __device__ __noinline__ void span_end(unsigned long long *span) {
 template <int P, int RECON, bool DAG, int KIND, bool SS>
 __device__ __forceinline__ void dslash_body(const DslashArgs &a);
 template <int P, int RECON, bool DAG, int KIND, bool SS>
-__global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF(P)) dslash_kernel(const __grid_constant__ DslashArgs a) {
+__global__ void __launch_bounds__(QX_DSLASH_THREADS, QX_MINB_OF2(P, RECON)) dslash_kernel(const __grid_constant__ DslashArgs a) {
 #ifndef QX_SPAN
 #define QX_SPAN 1
 #endif
