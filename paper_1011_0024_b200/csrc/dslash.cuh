@@ -474,11 +474,18 @@ template <int P> struct DslashMinBlocks { static constexpr int value = (P == 8) 
 #ifndef QX_R8_MINB_F16
 #define QX_R8_MINB_F16 6
 #endif
+// half recon-18 (both hops' raw operands in flight, dslash_pair) spills 150-180 B at 7 CTAs
+#ifndef QX_R18_MINB_F16
+#define QX_R18_MINB_F16 6
+#endif
 #ifdef QX_DSLASH_MINB
 #define QX_MINB_OF2(P, RECON) QX_DSLASH_MINB
 #else
-#define QX_MINB_OF2(P, RECON) \
-    ((RECON) == 8 && (P) == 4 ? QX_R8_MINB_F32 : ((RECON) == 8 && (P) == 2 ? QX_R8_MINB_F16 : DslashMinBlocks<P>::value))
+#define QX_MINB_OF2(P, RECON)                                                               \
+    ((RECON) == 8 && (P) == 4                                                               \
+         ? QX_R8_MINB_F32                                                                   \
+         : ((RECON) == 8 && (P) == 2 ? QX_R8_MINB_F16                                       \
+                                     : ((RECON) == 18 && (P) == 2 ? QX_R18_MINB_F16 : DslashMinBlocks<P>::value)))
 #endif
 // L1 prefetch (QX_RED_PF: the fused reduction's second operand, see dslash_site)
 __device__ __forceinline__ void pf_l1(const void *p) { asm volatile("prefetch.global.L1 [%0];" ::"l"(p)); }
